@@ -1,0 +1,80 @@
+"""Independent reference computations used to PIN the oracle (tests only).
+
+None of these shares code with oracle/ or with the product package; each is a
+different formulation of what the paper defines:
+
+* brute_local(): exhaustive enumeration of every local alignment (PAPER.md
+  L127-136: score of an alignment = sum of its columns; the similarity is the
+  maximal score) with affine gap runs costing Gs + k*Ge (Eqs. (3)-(4),
+  L185-194; reading R-1).  An alignment of two substrings is an
+  increasing chain of aligned pairs (i1<i2<..., j1<j2<...); between two
+  consecutive pairs the skipped query residues form one gap run and the skipped
+  subject residues another (interleaving them into more runs only adds opening
+  costs).  Leading/trailing gaps never help, the empty alignment scores 0.
+  The number of chains is C(m+n, m), so this is for m, n <= ~8.
+* linear_sw(): Eq. (1) (L159-165) with a constant gap g, full (m+1)x(n+1)
+  matrix -- the Gs = 0 special case of Eqs. (2)-(4).
+* ungapped_best(): max over diagonals of the maximal-sum segment (Kadane) --
+  what Eqs. (2)-(4) reduce to when every gap costs more than any alignment
+  could gain.
+* score_alignment(): score of a GIVEN alignment (two gapped strings of equal
+  length), the sec. II.A definition (L127-134), for the Fig. 1 worked example.
+"""
+from __future__ import annotations
+
+
+def brute_local(q, d, S, gs: int, ge: int) -> int:
+    m, n = len(q), len(d)
+
+    def gap(k: int) -> int:
+        return gs + k * ge if k > 0 else 0
+
+    best = 0
+    stack = [(i, j, int(S[q[i]][d[j]])) for i in range(m) for j in range(n)]
+    while stack:
+        i, j, sc = stack.pop()
+        if sc > best:
+            best = sc
+        for i2 in range(i + 1, m):
+            gi = gap(i2 - i - 1)
+            for j2 in range(j + 1, n):
+                stack.append((i2, j2, sc - gi - gap(j2 - j - 1) + int(S[q[i2]][d[j2]])))
+    return best
+
+
+def linear_sw(q, d, S, g: int) -> int:
+    """Eq. (1): H_ij = max(H_{i-1,j-1} + S_ij, H_{i,j-1} + g, H_{i-1,j} + g, 0); g <= 0."""
+    m, n = len(q), len(d)
+    H = [[0] * (n + 1) for _ in range(m + 1)]
+    best = 0
+    for i in range(1, m + 1):
+        for j in range(1, n + 1):
+            H[i][j] = max(H[i - 1][j - 1] + int(S[q[i - 1]][d[j - 1]]), H[i][j - 1] + g, H[i - 1][j] + g, 0)
+            best = max(best, H[i][j])
+    return best
+
+
+def ungapped_best(q, d, S) -> int:
+    m, n = len(q), len(d)
+    best = 0
+    for off in range(-(m - 1), n):
+        run = 0
+        for i in range(m):
+            j = i + off
+            if 0 <= j < n:
+                run = max(0, run + int(S[q[i]][d[j]]))
+                best = max(best, run)
+    return best
+
+
+def score_alignment(top: str, bottom: str, ma: int, mi: int, g: int) -> int:
+    assert len(top) == len(bottom)
+    s = 0
+    for a, b in zip(top, bottom):
+        if a == "-" or b == "-":
+            s += g
+        elif a == b:
+            s += ma
+        else:
+            s += mi
+    return s

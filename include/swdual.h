@@ -1,0 +1,165 @@
+/*
+ * swdual.h -- C ABI of the B200-native SWDUAL hot path.
+ *
+ * Computes, for a set of queries and a database of sequences, the
+ * Smith-Waterman local-alignment score with affine gaps (Gotoh) of every
+ * (query, database sequence) pair -- the computation the SWDUAL scheduler of
+ * Kedad-Sidhoum et al., ICPP 2014 distributes over CPUs and GPUs.
+ * PAPER.md = /root/reference/PAPER.md; citations give line numbers there.
+ *
+ *   "compare a set q of m query sequences to a set d of n database
+ *    sequences"                                         (L196-201, sec. II.C)
+ *   H_ij = max(H_{i-1,j-1} + S_ij, E_ij, F_ij, 0)              (Eq. (2))
+ *   E_ij = -Ge + max(E_{i,j-1}, H_{i,j-1} - Gs)                 (Eq. (3))
+ *   F_ij = -Ge + max(F_{i-1,j}, H_{i-1,j} - Gs)                 (Eq. (4))
+ *   first row and column of H are zero                           (L153-154)
+ *   result = the maximal score, "the similarity"                  (L135-136)
+ *
+ * so a gap of k residues costs gap_open + k * gap_extend (Gs + k*Ge).
+ *
+ * Conventions for every entry point:
+ *   - return int32 status: SW_OK (0) or a negative SW_E* code; no exception
+ *     crosses the ABI; sw_last_error() describes the last failure of a handle.
+ *   - "host" pointers are read/written by the CPU; "host or device" pointers
+ *     may be either (cudaPointerGetAttributes decides); the caller owns all
+ *     buffers it passes in and may free them when the call returns.
+ *   - a handle is bound to one CUDA device and is not thread-safe: one call at
+ *     a time per handle.
+ *   - cuda_stream is a cudaStream_t (NULL = legacy default stream).
+ */
+#ifndef SWDUAL_H
+#define SWDUAL_H
+
+#include <stdint.h>
+
+#ifdef __cplusplus
+extern "C" {
+#endif
+
+typedef struct sw_handle_s* sw_handle_t; /* opaque; bound to one CUDA device   */
+typedef struct sw_db_s* sw_db_t;         /* opaque; packed, device-resident DB  */
+
+enum {
+  SW_OK = 0,
+  SW_EINVAL = -1,       /* bad argument (null pointer, code >= alphabet, ...) */
+  SW_ENOMEM = -2,       /* device or host allocation failed                    */
+  SW_ECUDA = -3,        /* a CUDA call failed (message in sw_last_error)       */
+  SW_ESTATE = -4,       /* object used with the wrong handle / after free      */
+  SW_EUNSUPPORTED = -5  /* valid request outside what this build supports      */
+};
+
+enum { SW_FLAG_TIMING = 1 }; /* sw_init flags: record CUDA events around kernels */
+
+/* Create a handle on CUDA device `device`.  flags: SW_FLAG_* bits. */
+int32_t sw_init(int32_t device, uint32_t flags, sw_handle_t* out);
+
+/*
+ * Pack and upload a database (host packer; the paper's
+ * random-access binary format, L529-539).
+ *   codes       host, residue codes, codes[offsets[d] .. offsets[d+1]) is
+ *               sequence d; every code must be < alphabet_size.
+ *   offsets     host, int64[n_seqs + 1], non-decreasing, offsets[0] may be > 0.
+ *   n_seqs      >= 0; sequences of length 0 are allowed and score 0.
+ *   alphabet_size  1..32; code alphabet_size is used internally as PAD.
+ *   out         receives the DB; free with sw_free_db (or sw_free).
+ * The inputs are copied; the call returns when the upload is complete.
+ * Errors: SW_EINVAL (null pointer, bad offsets, code >= alphabet_size,
+ * alphabet_size out of range), SW_ENOMEM, SW_ECUDA.
+ */
+int32_t sw_load_db(sw_handle_t h, const uint8_t* codes, const int64_t* offsets, int64_t n_seqs,
+                   int32_t alphabet_size, void* cuda_stream, sw_db_t* out);
+
+/*
+ * Score every (query, database sequence) pair.
+ *   q_codes, q_offsets   host, queries in the same layout as sw_load_db
+ *                        (int64 q_offsets[n_queries + 1]); codes < alphabet.
+ *   matrix      host, int8[alphabet_size * alphabet_size], row-major,
+ *               matrix[a * alphabet_size + b] = S(query letter a, db letter b)
+ *               (S_ij scores query element i vs element j).
+ *   gap_open    Gs >= 0;  gap_extend  Ge >= 0;  Gs + Ge <= 32767.
+ *   scores      host or device, int32[n_queries][n_seqs], row-major, in the
+ *               caller's database order (the packer's length sort is undone).
+ * Device `scores`: the call is stream-ordered on cuda_stream; the caller
+ * synchronizes.  Host `scores`: the call returns after the results are copied.
+ * Exactness: scores are exact int32; the int16 DPX path flags any pair whose
+ * maximum reaches 32767 - max(matrix) and re-scores it in int32.
+ * Errors: SW_EINVAL, SW_ESTATE (db from another handle), SW_ENOMEM, SW_ECUDA.
+ * n_queries == 0 or an empty DB is valid and writes nothing.
+ */
+int32_t sw_search(sw_handle_t h, const uint8_t* q_codes, const int64_t* q_offsets, int32_t n_queries,
+                  sw_db_t db, const int8_t* matrix, int32_t gap_open, int32_t gap_extend, int32_t* scores,
+                  void* cuda_stream);
+
+int32_t sw_free_db(sw_db_t db);
+int32_t sw_free(sw_handle_t h); /* frees the handle and any DBs still attached */
+
+/* Message for the last failing call on h (or of the calling thread if h is NULL). */
+const char* sw_last_error(sw_handle_t h);
+
+/* --- introspection / tuning (not needed for plain use) ------------------- */
+
+typedef struct {
+  int64_t n_seqs, n_residues, n_pairs, n_long_pairs, max_len;
+  int32_t alphabet_size, device;
+} sw_db_info_t;
+int32_t sw_db_info(sw_db_t db, sw_db_info_t* out);
+
+typedef struct {
+  double cells;            /* sum_q m_q * sum_d n_d of the last search (real residues) */
+  double cells_computed;   /* including row/column padding and wavefront fill         */
+  double kernel_ms;        /* summed CUDA-event time of the scoring kernels (TIMING)   */
+  int32_t n_launches;      /* kernels launched by the last search                     */
+  int32_t n_score_launches;/* of which scoring (inter-task) kernels                   */
+  int32_t n_overflow;      /* pairs re-scored in int32 (needs a synchronize)           */
+  int32_t timing_valid;
+} sw_stats_t;
+/* Stats of the last sw_search; synchronizes the last search's stream. */
+int32_t sw_last_stats(sw_handle_t h, sw_stats_t* out);
+
+/*
+ * Integer options (testing / tuning).  Keys:
+ *   "overflow_threshold"  force the int16 re-score threshold (0 = automatic)
+ *   "force_G", "force_R"  force the inter-task lane-group geometry (0 = auto)
+ *   "timing"              1/0, same as SW_FLAG_TIMING
+ */
+int32_t sw_set_option(sw_handle_t h, const char* key, int64_t value);
+
+/* ASCII -> NCBI protein codes "ARNDCQEGHILKMFPSTWYVBZX*" (lower case folded, unknown -> X). */
+int32_t sw_encode_ascii(const char* s, int64_t n, uint8_t* out);
+
+/*
+ * Dual-approximation placement (sec. III): n_tasks tasks,
+ * task j takes p_cpu[j] on a CPU-type PE and p_gpu[j] on a GPU-type PE
+ * (host arrays, >= 0).  n_cpu >= 0 CPU PEs, n_gpu >= 0 GPU PEs, n_cpu+n_gpu >= 1.
+ * Binary search on the guess lambda (L468-481); per guess: greedy knapsack by
+ * decreasing p_cpu/p_gpu filling the GPUs up to area k*lambda (L370-387), the
+ * rest on CPUs, list scheduling on each side (L388-396); "NO" when the CPU area
+ * exceeds m*lambda.  out_pe[j] (host, int32[n_tasks]) = PE index, CPUs first
+ * (0..n_cpu-1) then GPUs (n_cpu..n_cpu+n_gpu-1).  out_makespan / out_lambda may
+ * be NULL.  Makespan <= 2 * lambda (Proposition 1).
+ */
+int32_t sw_schedule_dual(int64_t n_tasks, const double* p_cpu, const double* p_gpu, int32_t n_cpu,
+                         int32_t n_gpu, int32_t* out_pe, double* out_makespan, double* out_lambda);
+
+/*
+ * Host packer only (no device work): the packed form sw_load_db uploads.
+ * Non-empty sequences sorted by length (longest first, ties by index), paired
+ * neighbours (id1 = -1 for an odd leftover), each pair interleaved into 16-bit
+ * words code(id0) | code(id1) << 8 over `len` columns (multiple of 4, PAD =
+ * alphabet_size), pair p at stream[off .. off+len).  Pairs [0, n_long) are
+ * longer than t_long.  Two-phase: pass pairs == NULL and stream == NULL to get
+ * *n_pairs and *stream_words, then call again with buffers of those sizes.
+ * Errors: SW_EINVAL as for sw_load_db.
+ */
+typedef struct {
+  int64_t off;
+  int32_t len, id0, id1, pad_;
+} sw_pair_t;
+int32_t sw_pack_db_host(const uint8_t* codes, const int64_t* offsets, int64_t n_seqs, int32_t alphabet_size,
+                        int64_t t_long, sw_pair_t* pairs, int64_t* n_pairs, uint16_t* stream,
+                        int64_t* stream_words, int64_t* n_long);
+
+#ifdef __cplusplus
+}
+#endif
+#endif /* SWDUAL_H */

@@ -1,0 +1,156 @@
+"""Python API over the C ABI (include/swdual.h): same names, marshalling only.
+
+    h  = Handle(device=0)
+    db = h.load_db(codes, offsets, alphabet_size=24)        # sw_load_db
+    S  = h.search(q_codes, q_offsets, db, blosum62(), 10, 2) # sw_search -> int32[Q, N]
+
+PyTorch supplies device memory (output tensors) and streams; every score is
+computed by the library's CUDA kernels.
+"""
+from __future__ import annotations
+
+import ctypes
+
+import numpy as np
+
+from ._lib import DbInfo, Stats, SW_FLAG_TIMING, check, lib
+
+try:  # torch is plumbing only (device buffers, streams)
+    import torch
+except Exception:  # pragma: no cover
+    torch = None
+
+
+def _host(a, dtype) -> np.ndarray:
+    if torch is not None and isinstance(a, torch.Tensor):
+        a = a.detach().cpu().numpy()
+    return np.ascontiguousarray(np.asarray(a, dtype=dtype))
+
+
+def _vp(a: np.ndarray):
+    return a.ctypes.data_as(ctypes.c_void_p)
+
+
+def _stream_ptr(stream):
+    if stream is None:
+        if torch is not None and torch.cuda.is_available():
+            return ctypes.c_void_p(torch.cuda.current_stream().cuda_stream)
+        return ctypes.c_void_p(0)
+    if torch is not None and isinstance(stream, torch.cuda.Stream):
+        return ctypes.c_void_p(stream.cuda_stream)
+    return ctypes.c_void_p(int(stream))
+
+
+class Database:
+    """A packed, device-resident database (sw_db_t)."""
+
+    def __init__(self, handle: "Handle", ptr: ctypes.c_void_p, n_seqs: int):
+        self.handle = handle
+        self.ptr = ptr
+        self.n_seqs = n_seqs
+
+    def info(self) -> dict:
+        out = DbInfo()
+        check(lib().sw_db_info(self.ptr, ctypes.byref(out)), self.handle.ptr)
+        return {f: getattr(out, f) for f, _ in DbInfo._fields_}
+
+    def free(self) -> None:
+        if self.ptr:
+            lib().sw_free_db(self.ptr)
+            self.ptr = None
+
+
+class Handle:
+    """sw_handle_t bound to one CUDA device."""
+
+    def __init__(self, device: int = 0, timing: bool = False):
+        self.ptr = ctypes.c_void_p()
+        check(lib().sw_init(int(device), SW_FLAG_TIMING if timing else 0, ctypes.byref(self.ptr)))
+        self.device = int(device)
+        self._dbs: list[Database] = []
+
+    def set_option(self, key: str, value: int) -> None:
+        check(lib().sw_set_option(self.ptr, key.encode(), int(value)), self.ptr)
+
+    def load_db(self, codes, offsets, alphabet_size: int = 24, stream=None) -> Database:
+        codes = _host(codes, np.uint8)
+        offsets = _host(offsets, np.int64)
+        n = len(offsets) - 1
+        out = ctypes.c_void_p()
+        check(lib().sw_load_db(self.ptr, _vp(codes) if codes.size else None, _vp(offsets), n, int(alphabet_size),
+                               _stream_ptr(stream), ctypes.byref(out)), self.ptr)
+        db = Database(self, out, n)
+        self._dbs.append(db)
+        return db
+
+    def search(self, q_codes, q_offsets, db: Database, matrix, gap_open: int = 10, gap_extend: int = 2,
+               out=None, stream=None):
+        """int32 scores[Q][N] in the caller's DB order.
+
+        out: None -> a new torch.int32 CUDA tensor (stream-ordered) if torch has CUDA, else a numpy array;
+             a torch CUDA tensor -> written in place on `stream` (caller synchronizes);
+             a numpy array -> host output, returned after the copy completes.
+        """
+        q_codes = _host(q_codes, np.uint8)
+        q_offsets = _host(q_offsets, np.int64)
+        matrix = _host(matrix, np.int8)
+        nq = len(q_offsets) - 1
+        N = db.n_seqs
+        if out is None:
+            if torch is not None and torch.cuda.is_available():
+                out = torch.empty((nq, N), dtype=torch.int32, device=f"cuda:{self.device}")
+            else:
+                out = np.zeros((nq, N), dtype=np.int32)
+        if torch is not None and isinstance(out, torch.Tensor):
+            assert out.dtype == torch.int32 and out.is_contiguous() and tuple(out.shape) == (nq, N)
+            optr = ctypes.c_void_p(out.data_ptr())
+        else:
+            assert out.dtype == np.int32 and out.flags.c_contiguous and out.shape == (nq, N)
+            optr = _vp(out)
+        check(lib().sw_search(self.ptr, _vp(q_codes) if q_codes.size else None, _vp(q_offsets), nq, db.ptr,
+                              _vp(matrix), int(gap_open), int(gap_extend), optr, _stream_ptr(stream)), self.ptr)
+        return out
+
+    def last_stats(self) -> dict:
+        s = Stats()
+        check(lib().sw_last_stats(self.ptr, ctypes.byref(s)), self.ptr)
+        return {f: getattr(s, f) for f, _ in Stats._fields_}
+
+    def close(self) -> None:
+        if self.ptr:
+            lib().sw_free(self.ptr)
+            self.ptr = None
+            for d in self._dbs:
+                d.ptr = None
+
+    def __enter__(self):
+        return self
+
+    def __exit__(self, *exc):
+        self.close()
+
+    def __del__(self):
+        try:
+            self.close()
+        except Exception:
+            pass
+
+
+def encode_ascii(s: str) -> np.ndarray:
+    """sw_encode_ascii: protein string -> NCBI codes (unknown -> X)."""
+    b = s.encode("ascii", "replace")
+    out = np.zeros(len(b), dtype=np.uint8)
+    check(lib().sw_encode_ascii(b, len(b), _vp(out) if len(b) else None))
+    return out
+
+
+def schedule_dual(p_cpu, p_gpu, n_cpu: int, n_gpu: int):
+    """sw_schedule_dual: (pe int32[n], makespan, lambda); PEs 0..n_cpu-1 are CPUs, then GPUs."""
+    pc = _host(p_cpu, np.float64)
+    pg = _host(p_gpu, np.float64)
+    n = len(pc)
+    pe = np.full(n, -1, dtype=np.int32)
+    mk, lam = ctypes.c_double(), ctypes.c_double()
+    check(lib().sw_schedule_dual(n, _vp(pc) if n else None, _vp(pg) if n else None, int(n_cpu), int(n_gpu),
+                                 _vp(pe) if n else None, ctypes.byref(mk), ctypes.byref(lam)))
+    return pe, mk.value, lam.value

@@ -1,0 +1,532 @@
+// Host engine and C ABI of the SWDUAL hot path (include/swdual.h).
+//
+//   sw_load_db : host packer -- validate codes, sort the
+//                database by length (longest first, ties by index), pair
+//                neighbours, interleave each pair column by column into 16-bit
+//                words padded to 4 columns, upload stream + pair table once.
+//   sw_search  : per query, build the int8 query profile on the device, launch
+//                the inter-task DPX kernel over the short pairs and over the
+//                long pairs, then the int32 re-score of flagged pairs; scores
+//                land directly in the caller's DB order (un-permute fused into
+//                the kernel epilogue).
+#include <algorithm>
+#include <atomic>
+#include <cstdio>
+#include <cstring>
+#include <mutex>
+#include <new>
+#include <stdexcept>
+#include <numeric>
+#include <string>
+#include <thread>
+#include <vector>
+
+#include <cuda_runtime.h>
+
+#include "../../include/swdual.h"
+#include "sw_internal.h"
+
+using namespace swdual;
+
+namespace {
+
+thread_local std::string g_tls_err;
+
+struct DevBuf {
+  void* p = nullptr;
+  size_t n = 0;
+  DevBuf() = default;
+  DevBuf(const DevBuf&) = delete;
+  DevBuf& operator=(const DevBuf&) = delete;
+  ~DevBuf() { release(); }
+  void release() {
+    if (p) cudaFree(p);
+    p = nullptr;
+    n = 0;
+  }
+  cudaError_t ensure(size_t bytes) {
+    if (bytes <= n && p) return cudaSuccess;
+    release();
+    size_t b = std::max<size_t>(bytes, 256);
+    cudaError_t e = cudaMalloc(&p, b);
+    if (e != cudaSuccess) { p = nullptr; return e; }
+    n = b;
+    return cudaSuccess;
+  }
+  template <class T> T* as() const { return reinterpret_cast<T*>(p); }
+};
+
+struct SwError {
+  int32_t code;
+  std::string msg;
+};
+
+#define SW_CK(call)                                                                          \
+  do {                                                                                       \
+    cudaError_t e_ = (call);                                                                 \
+    if (e_ != cudaSuccess)                                                                   \
+      throw SwError{e_ == cudaErrorMemoryAllocation ? SW_ENOMEM : SW_ECUDA,                  \
+                    std::string(#call) + ": " + cudaGetErrorString(e_)};                     \
+  } while (0)
+
+[[noreturn]] void fail(int32_t code, const std::string& m) { throw SwError{code, m}; }
+
+constexpr int T_LONG = 3000;  // pairs longer than this are launched separately
+
+}  // namespace
+
+struct sw_db_s;
+
+struct sw_handle_s {
+  int device = 0;
+  int sms = 148;
+  uint32_t flags = 0;
+  std::string err;
+  std::vector<sw_db_s*> dbs;
+  // scratch (grown on demand)
+  DevBuf qcodes, qoff, matrix, prof, bbuf, counters, ovf, ovf_count, scores_tmp, rbuf;
+  // options
+  int64_t opt_thr = 0, opt_G = 0, opt_R = 0;
+  // last-search bookkeeping
+  sw_stats_t stats{};
+  cudaStream_t last_stream = nullptr;
+  std::vector<std::pair<cudaEvent_t, cudaEvent_t>> events;
+  size_t n_events_used = 0;
+};
+
+struct sw_db_s {
+  sw_handle_s* h = nullptr;
+  int64_t n_seqs = 0, n_res = 0;
+  int alpha = 0;
+  int64_t max_len = 0;
+  std::vector<PairRec> pairs;    // host copy, sorted longest first
+  std::vector<int64_t> seq_len;  // caller order
+  std::vector<int64_t> sorted_lens;  // descending, non-empty only (for overflow bounds)
+  int n_long = 0;                // pairs [0, n_long) have len > T_LONG
+  DevBuf stream, dpairs;
+};
+
+static int32_t set_err(sw_handle_s* h, int32_t code, const std::string& m) {
+  if (h) h->err = m;
+  g_tls_err = m;
+  return code;
+}
+
+template <class F>
+static int32_t guarded(sw_handle_s* h, F&& f) {
+  try {
+    f();
+    return SW_OK;
+  } catch (const SwError& e) {
+    return set_err(h, e.code, e.msg);
+  } catch (const std::bad_alloc&) {
+    return set_err(h, SW_ENOMEM, "host allocation failed");
+  } catch (const std::exception& e) {
+    return set_err(h, SW_EINVAL, e.what());
+  }
+}
+
+// ----------------------------------------------------------------------------
+// geometry of the inter-task kernel for a query of m rows and a launch whose
+// pairs average Lavg columns
+static ProfGeom make_geom(int G, int R, int m, int alpha) {
+  ProfGeom g{};
+  g.G = G;
+  g.R = R;
+  g.LB = ((R % 8 == 0) ? (((R / 8) | 1) * 8) : (((R / 4) | 1) * 4));
+  g.LS = G * g.LB;
+  g.NL = alpha + 1;
+  g.SB = ((g.NL * g.LS + 15) / 16) * 16;
+  g.n_strips = std::max(1, (m + G * R - 1) / (G * R));
+  return g;
+}
+
+static void choose_geom(const sw_handle_s* h, int m, double Lavg, bool long_pairs, int& G, int& R) {
+  if (h->opt_G > 0 && h->opt_R > 0) {
+    G = int(h->opt_G);
+    R = int(h->opt_R);
+    return;
+  }
+  static const int Gs[] = {4, 8, 16, 32};
+  static const int Rs[] = {8, 12, 16, 20, 24, 28, 32};
+  double best = 1e300;
+  G = 32;
+  R = 16;
+  for (int g : Gs) {
+    if (long_pairs && g != 32) continue;
+    for (int r : Rs) {
+      const int strips = std::max(1, (m + g * r - 1) / (g * r));
+      const double rows = double(strips) * g * r;
+      // per-step overhead ~ 7 instr / (5.5 per row) plus register-pressure penalty for big R
+      const double per_cell = 1.0 + 7.0 / (5.5 * r) + (r > 24 ? 0.06 : 0.0);
+      const double strip_ovh = strips > 1 ? 0.02 : 0.0;
+      const double cost = rows * (Lavg + g) * per_cell * (1.0 + strip_ovh);
+      if (cost < best) { best = cost; G = g; R = r; }
+    }
+  }
+}
+
+// ----------------------------------------------------------------------------
+extern "C" {
+
+int32_t sw_init(int32_t device, uint32_t flags, sw_handle_t* out) {
+  if (!out) return set_err(nullptr, SW_EINVAL, "sw_init: out is NULL");
+  *out = nullptr;
+  sw_handle_s* h = nullptr;
+  int32_t rc = guarded(nullptr, [&] {
+    int n = 0;
+    SW_CK(cudaGetDeviceCount(&n));
+    if (device < 0 || device >= n) fail(SW_EINVAL, "sw_init: bad device index");
+    SW_CK(cudaSetDevice(device));
+    h = new sw_handle_s();
+    h->device = device;
+    h->flags = flags;
+    SW_CK(cudaDeviceGetAttribute(&h->sms, cudaDevAttrMultiProcessorCount, device));
+  });
+  if (rc != SW_OK) {
+    delete h;
+    return rc;
+  }
+  *out = h;
+  return SW_OK;
+}
+
+int32_t sw_set_option(sw_handle_t h, const char* key, int64_t value) {
+  if (!h || !key) return set_err(h, SW_EINVAL, "sw_set_option: NULL argument");
+  std::string k(key);
+  if (k == "overflow_threshold") h->opt_thr = value;
+  else if (k == "force_G") {
+    if (value != 0 && value != 4 && value != 8 && value != 16 && value != 32)
+      return set_err(h, SW_EINVAL, "force_G must be 0, 4, 8, 16 or 32");
+    h->opt_G = value;
+  } else if (k == "force_R") {
+    if (value != 0 && (value < 8 || value > 32 || value % 4))
+      return set_err(h, SW_EINVAL, "force_R must be 0 or a multiple of 4 in [8, 32]");
+    h->opt_R = value;
+  } else if (k == "timing") {
+    if (value) h->flags |= SW_FLAG_TIMING; else h->flags &= ~uint32_t(SW_FLAG_TIMING);
+  } else
+    return set_err(h, SW_EINVAL, "sw_set_option: unknown key " + k);
+  return SW_OK;
+}
+
+int32_t sw_load_db(sw_handle_t h, const uint8_t* codes, const int64_t* offsets, int64_t n_seqs,
+                   int32_t alphabet_size, void* cuda_stream, sw_db_t* out) {
+  if (!h) return set_err(nullptr, SW_EINVAL, "sw_load_db: handle is NULL");
+  if (!out) return set_err(h, SW_EINVAL, "sw_load_db: out is NULL");
+  *out = nullptr;
+  sw_db_s* db = nullptr;
+  int32_t rc = guarded(h, [&] {
+    SW_CK(cudaSetDevice(h->device));
+    cudaStream_t st = reinterpret_cast<cudaStream_t>(cuda_stream);
+    db = new sw_db_s();
+    db->h = h;
+    db->n_seqs = n_seqs;
+    db->alpha = alphabet_size;
+    Packed P;
+    try {
+      pack_db(codes, offsets, n_seqs, alphabet_size, T_LONG, P);
+    } catch (const std::invalid_argument& e) {
+      fail(SW_EINVAL, std::string("sw_load_db: ") + e.what());
+    }
+    db->n_res = P.n_res;
+    db->max_len = P.max_len;
+    db->n_long = P.n_long;
+    db->pairs = std::move(P.pairs);
+    db->seq_len = std::move(P.seq_len);
+    db->sorted_lens = std::move(P.sorted_lens);
+    const size_t np = db->pairs.size();
+    std::vector<uint16_t>& stream = P.stream;
+    SW_CK(db->stream.ensure(stream.size() * sizeof(uint16_t)));
+    SW_CK(db->dpairs.ensure(std::max<size_t>(np, 1) * sizeof(PairRec)));
+    SW_CK(cudaMemcpyAsync(db->stream.p, stream.data(), stream.size() * sizeof(uint16_t), cudaMemcpyHostToDevice, st));
+    if (np)
+      SW_CK(cudaMemcpyAsync(db->dpairs.p, db->pairs.data(), np * sizeof(PairRec), cudaMemcpyHostToDevice, st));
+    SW_CK(cudaStreamSynchronize(st));
+  });
+  if (rc != SW_OK) {
+    delete db;
+    return rc;
+  }
+  h->dbs.push_back(db);
+  *out = db;
+  return SW_OK;
+}
+
+int32_t sw_db_info(sw_db_t db, sw_db_info_t* out) {
+  if (!db || !out) return set_err(nullptr, SW_EINVAL, "sw_db_info: NULL argument");
+  out->n_seqs = db->n_seqs;
+  out->n_residues = db->n_res;
+  out->n_pairs = int64_t(db->pairs.size());
+  out->n_long_pairs = db->n_long;
+  out->max_len = db->max_len;
+  out->alphabet_size = db->alpha;
+  out->device = db->h ? db->h->device : -1;
+  return SW_OK;
+}
+
+static cudaEvent_t* next_event_pair(sw_handle_s* h) {
+  if (h->n_events_used == h->events.size()) {
+    cudaEvent_t a, b;
+    if (cudaEventCreate(&a) != cudaSuccess) return nullptr;
+    if (cudaEventCreate(&b) != cudaSuccess) { cudaEventDestroy(a); return nullptr; }
+    h->events.push_back({a, b});
+  }
+  return &h->events[h->n_events_used++].first;
+}
+
+int32_t sw_search(sw_handle_t h, const uint8_t* q_codes, const int64_t* q_offsets, int32_t n_queries, sw_db_t db,
+                  const int8_t* matrix, int32_t gap_open, int32_t gap_extend, int32_t* scores, void* cuda_stream) {
+  if (!h) return set_err(nullptr, SW_EINVAL, "sw_search: handle is NULL");
+  return guarded(h, [&] {
+    if (!db) fail(SW_EINVAL, "sw_search: db is NULL");
+    if (db->h != h) fail(SW_ESTATE, "sw_search: db belongs to another handle");
+    if (n_queries < 0) fail(SW_EINVAL, "sw_search: n_queries < 0");
+    if (n_queries > 0 && !q_offsets) fail(SW_EINVAL, "sw_search: q_offsets is NULL");
+    if (!matrix) fail(SW_EINVAL, "sw_search: matrix is NULL");
+    if (gap_open < 0 || gap_extend < 0) fail(SW_EINVAL, "sw_search: gap penalties must be >= 0");
+    if (int64_t(gap_open) + gap_extend > 32767) fail(SW_EINVAL, "sw_search: gap_open + gap_extend > 32767");
+    const int alpha = db->alpha;
+    SW_CK(cudaSetDevice(h->device));
+    cudaStream_t st = reinterpret_cast<cudaStream_t>(cuda_stream);
+    h->stats = sw_stats_t{};
+    h->n_events_used = 0;
+    h->last_stream = st;
+    if (n_queries == 0 || db->n_seqs == 0) return;
+    if (!scores) fail(SW_EINVAL, "sw_search: scores is NULL");
+    // queries
+    std::vector<int64_t> qlen(static_cast<size_t>(n_queries));
+    int64_t qtot = 0;
+    for (int i = 0; i < n_queries; ++i) {
+      qlen[size_t(i)] = q_offsets[i + 1] - q_offsets[i];
+      if (qlen[size_t(i)] < 0) fail(SW_EINVAL, "sw_search: q_offsets not non-decreasing");
+      if (qlen[size_t(i)] > (int64_t(1) << 30)) fail(SW_EUNSUPPORTED, "sw_search: query longer than 2^30");
+      qtot += qlen[size_t(i)];
+    }
+    if (qtot > 0 && !q_codes) fail(SW_EINVAL, "sw_search: q_codes is NULL");
+    const uint8_t* qbase = q_codes ? q_codes + q_offsets[0] : nullptr;
+    for (int64_t i = 0; i < qtot; ++i)
+      if (qbase[i] >= alpha) fail(SW_EINVAL, "sw_search: query code >= alphabet_size");
+    int smax = -128;
+    for (int i = 0; i < alpha * alpha; ++i) smax = std::max<int>(smax, matrix[i]);
+    // int16 re-score threshold: flag if max >= 32767 - S_max
+    int32_t thr = smax > 0 ? 32767 - smax : 32768;
+    if (h->opt_thr > 0) thr = int32_t(h->opt_thr);
+    // output
+    cudaPointerAttributes pa{};
+    bool dev_scores = false;
+    if (cudaPointerGetAttributes(&pa, scores) == cudaSuccess)
+      dev_scores = (pa.type == cudaMemoryTypeDevice || pa.type == cudaMemoryTypeManaged);
+    cudaGetLastError();
+    const int64_t N = db->n_seqs;
+    const size_t out_bytes = size_t(n_queries) * size_t(N) * sizeof(int32_t);
+    int32_t* dscores = scores;
+    if (!dev_scores) {
+      SW_CK(h->scores_tmp.ensure(out_bytes));
+      dscores = h->scores_tmp.as<int32_t>();
+    }
+    // upload queries, offsets rebased to 0
+    std::vector<int64_t> qoff0(size_t(n_queries) + 1);
+    for (int i = 0; i <= n_queries; ++i) qoff0[size_t(i)] = q_offsets[i] - q_offsets[0];
+    SW_CK(h->qcodes.ensure(size_t(std::max<int64_t>(qtot, 1))));
+    SW_CK(h->qoff.ensure(qoff0.size() * sizeof(int64_t)));
+    SW_CK(h->matrix.ensure(size_t(alpha * alpha)));
+    if (qtot) SW_CK(cudaMemcpyAsync(h->qcodes.p, qbase, size_t(qtot), cudaMemcpyHostToDevice, st));
+    SW_CK(cudaMemcpyAsync(h->qoff.p, qoff0.data(), qoff0.size() * sizeof(int64_t), cudaMemcpyHostToDevice, st));
+    SW_CK(cudaMemcpyAsync(h->matrix.p, matrix, size_t(alpha * alpha), cudaMemcpyHostToDevice, st));
+    SW_CK(cudaMemsetAsync(dscores, 0, out_bytes, st));
+    int launches = 0;
+    // overflow list capacity: a pair can only be flagged if min(m, n) * S_max >= thr
+    int64_t ovf_cap = 0;
+    if (smax > 0) {
+      const int64_t need = (int64_t(thr) + smax - 1) / smax;  // min length that can reach thr
+      // sorted_lens is descending: count the DB sequences of length >= need
+      const int64_t nd_ge = std::lower_bound(db->sorted_lens.begin(), db->sorted_lens.end(), need,
+                                             [](int64_t v, int64_t x) { return v >= x; }) -
+                            db->sorted_lens.begin();
+      for (int i = 0; i < n_queries; ++i)
+        if (qlen[size_t(i)] >= need) ovf_cap += nd_ge;
+    }
+    if (ovf_cap > (int64_t(1) << 28)) fail(SW_EUNSUPPORTED, "sw_search: overflow list bound too large");
+    SW_CK(h->ovf.ensure(size_t(std::max<int64_t>(ovf_cap, 1)) * sizeof(OvfRec)));
+    SW_CK(h->ovf_count.ensure(sizeof(int)));
+    SW_CK(cudaMemsetAsync(h->ovf_count.p, 0, sizeof(int), st));
+    // work counters: 2 launches per query
+    SW_CK(h->counters.ensure(size_t(2 * n_queries) * sizeof(int)));
+    SW_CK(cudaMemsetAsync(h->counters.p, 0, size_t(2 * n_queries) * sizeof(int), st));
+    const bool timing = (h->flags & SW_FLAG_TIMING) != 0;
+    double cells_computed = 0;
+    const int np = int(db->pairs.size());
+    const int nlong = db->n_long;
+    // average pair length of the short and long ranges
+    double sum_short = 0, sum_long = 0;
+    int32_t max_short = 0, max_long = 0;
+    for (int p = 0; p < np; ++p) {
+      if (p < nlong) { sum_long += db->pairs[size_t(p)].len; max_long = std::max(max_long, db->pairs[size_t(p)].len); }
+      else { sum_short += db->pairs[size_t(p)].len; max_short = std::max(max_short, db->pairs[size_t(p)].len); }
+    }
+    const int nshort = np - nlong;
+    const uint32_t nGe16 = uint32_t(uint16_t(int16_t(-gap_extend)));
+    const uint32_t nGsGe16 = uint32_t(uint16_t(int16_t(-(gap_open + gap_extend))));
+    for (int qi = 0; qi < n_queries; ++qi) {
+      const int m = int(qlen[size_t(qi)]);
+      if (m == 0) continue;
+      for (int part = 0; part < 2; ++part) {
+        const bool lp = (part == 0);
+        const int pb = lp ? 0 : nlong, pe = lp ? nlong : np;
+        if (pe <= pb) continue;
+        const double Lavg = lp ? sum_long / nlong : sum_short / nshort;
+        const int32_t Lmax = lp ? max_long : max_short;
+        int G, R;
+        choose_geom(h, m, Lavg, lp, G, R);
+        if (!inter_config_supported(G, R)) fail(SW_EUNSUPPORTED, "no kernel for this geometry");
+        const ProfGeom geom = make_geom(G, R, m, alpha);
+        SW_CK(h->prof.ensure(size_t(geom.n_strips) * geom.SB));
+        SW_CK(launch_build_profile(h->qcodes.as<uint8_t>() + qoff0[size_t(qi)], m, h->matrix.as<int8_t>(), alpha,
+                                   geom, h->prof.as<uint8_t>(), st));
+        ++launches;
+        const int NT = 256, NG = NT / G;
+        const int smem = geom.SB;
+        const int occ = inter_max_ctas_per_sm(G, R, NT, smem);
+        if (occ <= 0) fail(SW_ECUDA, "inter kernel does not fit on an SM");
+        const int nchunks = (pe - pb + NG - 1) / NG;
+        const int grid = std::max(1, std::min(nchunks, occ * h->sms));
+        const int bcap = Lmax + G + 8;
+        if (geom.n_strips > 1) SW_CK(h->bbuf.ensure(size_t(grid) * NG * bcap * sizeof(uint2)));
+        InterArgs a{};
+        a.prof = h->prof.as<uint8_t>();
+        a.n_strips = geom.n_strips;
+        a.SB = geom.SB;
+        a.LS = geom.LS;
+        a.LB = geom.LB;
+        a.stream = db->stream.as<uint16_t>();
+        a.pairs = db->dpairs.as<PairRec>();
+        a.pair_begin = pb;
+        a.pair_end = pe;
+        a.bbuf = geom.n_strips > 1 ? h->bbuf.as<uint2>() : nullptr;
+        a.bcap = bcap;
+        a.work_counter = h->counters.as<int>() + 2 * qi + part;
+        a.scores = dscores + int64_t(qi) * N;
+        a.thr = thr;
+        a.ovf = h->ovf.as<OvfRec>();
+        a.ovf_count = h->ovf_count.as<int>();
+        a.ovf_cap = int(ovf_cap);
+        a.qidx = qi;
+        a.code_pad2 = uint32_t(alpha) | (uint32_t(alpha) << 8);
+        a.nGe = nGe16 | (nGe16 << 16);
+        a.nGsGe = nGsGe16 | (nGsGe16 << 16);
+        cudaEvent_t* ev = timing ? next_event_pair(h) : nullptr;
+        if (ev) SW_CK(cudaEventRecord(ev[0], st));
+        SW_CK(launch_inter(G, R, NT, grid, smem, a, st));
+        if (ev) SW_CK(cudaEventRecord(ev[1], st));
+        ++launches;
+        ++h->stats.n_score_launches;
+        double sumL = 0;
+        for (int p = pb; p < pe; ++p) sumL += db->pairs[size_t(p)].len + G;
+        cells_computed += 2.0 * sumL * double(geom.n_strips) * G * R;
+      }
+    }
+    if (ovf_cap > 0) {
+      int32_t Lmax = std::max(max_short, max_long);
+      const int grid = std::max(1, std::min<int>(int((ovf_cap + RESCORE_WARPS - 1) / RESCORE_WARPS), h->sms * 2));
+      const int bcap = Lmax + 40;
+      SW_CK(h->rbuf.ensure(size_t(grid) * RESCORE_WARPS * bcap * sizeof(int2)));
+      RescoreArgs r{};
+      r.qcodes = h->qcodes.as<uint8_t>();
+      r.qoff = h->qoff.as<int64_t>();
+      r.stream = db->stream.as<uint16_t>();
+      r.pairs = db->dpairs.as<PairRec>();
+      r.matrix = h->matrix.as<int8_t>();
+      r.alpha = alpha;
+      r.ovf = h->ovf.as<OvfRec>();
+      r.ovf_count = h->ovf_count.as<int>();
+      r.bbuf = h->rbuf.as<int2>();
+      r.bcap = bcap;
+      r.scores = dscores;
+      r.n_seqs = N;
+      r.Gs = gap_open;
+      r.Ge = gap_extend;
+      SW_CK(launch_rescore(grid, r, st));
+      ++launches;
+    }
+    if (!dev_scores) {
+      SW_CK(cudaMemcpyAsync(scores, dscores, out_bytes, cudaMemcpyDeviceToHost, st));
+      SW_CK(cudaStreamSynchronize(st));
+    }
+    double sq = 0;
+    for (auto L : qlen) sq += double(L);
+    h->stats.cells = sq * double(db->n_res);
+    h->stats.cells_computed = cells_computed;
+    h->stats.n_launches = launches;
+  });
+}
+
+int32_t sw_last_stats(sw_handle_t h, sw_stats_t* out) {
+  if (!h || !out) return set_err(h, SW_EINVAL, "sw_last_stats: NULL argument");
+  return guarded(h, [&] {
+    SW_CK(cudaSetDevice(h->device));
+    SW_CK(cudaStreamSynchronize(h->last_stream));
+    sw_stats_t s = h->stats;
+    if (h->ovf_count.p) {
+      int c = 0;
+      SW_CK(cudaMemcpy(&c, h->ovf_count.p, sizeof(int), cudaMemcpyDeviceToHost));
+      s.n_overflow = c;
+    }
+    double ms = 0;
+    for (size_t i = 0; i < h->n_events_used; ++i) {
+      float t = 0;
+      SW_CK(cudaEventElapsedTime(&t, h->events[i].first, h->events[i].second));
+      ms += t;
+    }
+    s.kernel_ms = ms;
+    s.timing_valid = h->n_events_used > 0 ? 1 : 0;
+    *out = s;
+  });
+}
+
+int32_t sw_free_db(sw_db_t db) {
+  if (!db) return SW_OK;
+  sw_handle_s* h = db->h;
+  if (h) {
+    cudaSetDevice(h->device);
+    auto it = std::find(h->dbs.begin(), h->dbs.end(), db);
+    if (it != h->dbs.end()) h->dbs.erase(it);
+  }
+  delete db;
+  return SW_OK;
+}
+
+int32_t sw_free(sw_handle_t h) {
+  if (!h) return SW_OK;
+  cudaSetDevice(h->device);
+  for (auto* db : h->dbs) {
+    db->h = nullptr;
+    delete db;
+  }
+  h->dbs.clear();
+  for (auto& e : h->events) {
+    cudaEventDestroy(e.first);
+    cudaEventDestroy(e.second);
+  }
+  delete h;
+  return SW_OK;
+}
+
+const char* sw_last_error(sw_handle_t h) { return h ? h->err.c_str() : g_tls_err.c_str(); }
+
+int32_t sw_encode_ascii(const char* s, int64_t n, uint8_t* out) {
+  static const char* AL = "ARNDCQEGHILKMFPSTWYVBZX*";
+  if (n < 0 || (n > 0 && (!s || !out))) return set_err(nullptr, SW_EINVAL, "sw_encode_ascii: bad argument");
+  uint8_t lut[256];
+  std::memset(lut, 22, sizeof(lut));  // X
+  for (int k = 0; k < 24; ++k) {
+    lut[uint8_t(AL[k])] = uint8_t(k);
+    if (AL[k] >= 'A' && AL[k] <= 'Z') lut[uint8_t(AL[k] - 'A' + 'a')] = uint8_t(k);
+  }
+  lut[uint8_t('U')] = lut[uint8_t('u')] = 4;   // selenocysteine -> C
+  lut[uint8_t('O')] = lut[uint8_t('o')] = 11;  // pyrrolysine -> K
+  for (int64_t i = 0; i < n; ++i) out[i] = lut[uint8_t(s[i])];
+  return SW_OK;
+}
+
+}  // extern "C"

@@ -1,0 +1,315 @@
+// SWDUAL hot-path kernels for sm_100a: query-profile build, the inter-task
+// s16x2 DPX scoring kernel and the exact int32 re-score kernel.
+//
+// Inter-task kernel (the paper's "very coarse-grained" split
+// across workers, with the "fine-grained" wavefront inside a
+// worker, L202-216 / Fig. 2):
+//   * a lane GROUP of G lanes scores one database pair (two length-neighbours,
+//     one per s16x2 half) against one query;
+//   * lane k of the group owns R consecutive query rows of the current strip
+//     (strip height G*R rows); at step t it computes column t-k, so the group
+//     sweeps the matrix as an anti-diagonal wave: the bottom row (H, F) and the
+//     residue codes travel one lane down per step over warp shuffles;
+//   * queries taller than one strip are done in passes; the last lane writes the
+//     strip's bottom row to a per-group global boundary row that lane 0 reads
+//     in the next pass;
+//   * the int8 query profile of the current strip sits in shared memory;
+//   * CTAs are persistent and take chunks of NT/G pairs from an atomic counter,
+//     pairs sorted longest first.
+#include <cstdio>
+#include "sw_internal.h"
+#include "sw_device.cuh"
+
+namespace swdual {
+
+constexpr uint32_t FULL = 0xffffffffu;
+constexpr int8_t PAD_SCORE = -64;  // S[.][PAD] = S[PAD][.] <= 0 (reading R-12)
+
+// ---------------------------------------------------------------------------
+// Query profile: prof[s][a][k][r] = S[q[s*G*R + k*R + r]][a]  (int8)
+//   a < alpha: matrix column a; a == alpha: PAD; rows >= m: PAD.
+__global__ void build_profile_kernel(const uint8_t* __restrict__ q, int m, const int8_t* __restrict__ M,
+                                     int alpha, ProfGeom g, uint8_t* __restrict__ prof) {
+  const int64_t total = (int64_t)g.n_strips * g.SB;
+  for (int64_t i = blockIdx.x * (int64_t)blockDim.x + threadIdx.x; i < total;
+       i += (int64_t)gridDim.x * blockDim.x) {
+    const int s = int(i / g.SB);
+    const int rem = int(i - (int64_t)s * g.SB);
+    int8_t v = 0;
+    if (rem < g.NL * g.LS) {
+      const int a = rem / g.LS;
+      const int rr = rem - a * g.LS;
+      const int k = rr / g.LB;
+      const int r = rr - k * g.LB;
+      if (r < g.R) {
+        const int row = s * g.G * g.R + k * g.R + r;
+        v = (row < m && a < alpha) ? M[q[row] * alpha + a] : PAD_SCORE;
+      }
+    }
+    prof[i] = uint8_t(v);
+  }
+}
+
+cudaError_t launch_build_profile(const uint8_t* q, int m, const int8_t* matrix, int alpha, const ProfGeom& g,
+                                 uint8_t* prof, cudaStream_t st) {
+  const int64_t total = (int64_t)g.n_strips * g.SB;
+  int grid = int((total + 255) / 256);
+  if (grid > 4096) grid = 4096;
+  if (grid < 1) grid = 1;
+  build_profile_kernel<<<grid, 256, 0, st>>>(q, m, matrix, alpha, g, prof);
+  return cudaGetLastError();
+}
+
+// ---------------------------------------------------------------------------
+__device__ __forceinline__ void copy_strip(uint8_t* dst, const uint8_t* __restrict__ src, int bytes) {
+  const uint4* s = reinterpret_cast<const uint4*>(src);
+  uint4* d = reinterpret_cast<uint4*>(dst);
+  for (int i = threadIdx.x; i < bytes / 16; i += blockDim.x) d[i] = __ldg(s + i);
+}
+
+template <int G, int R>
+__device__ __forceinline__ void strip_pass(const InterArgs& a, const uint8_t* sprof, const PairRec& pr, int T,
+                                           int k, bool rd, bool wr, uint2* __restrict__ bb, uint32_t& best) {
+  uint32_t Hl[R], E[R];
+#pragma unroll
+  for (int r = 0; r < R; ++r) { Hl[r] = 0; E[r] = 0; }
+  uint32_t hdiag = 0, sH = 0, sF = 0, sC = a.code_pad2;
+  const uint2* __restrict__ codes = reinterpret_cast<const uint2*>(a.stream + pr.off);
+  const int L = pr.len;
+  const uint32_t pad4 = a.code_pad2 | (a.code_pad2 << 16);
+  const uint32_t laneoff = uint32_t(k) * a.LB;
+  const bool lead = (k == 0), tail = (k == G - 1);
+
+  // lane 0 prefetch of block 0: 4 columns of codes and (if rd) 4 boundary cells
+  uint2 cw = make_uint2(pad4, pad4);
+  uint2 tb0 = make_uint2(0, 0), tb1 = tb0, tb2 = tb0, tb3 = tb0;
+  if (lead) {
+    if (L > 0) cw = codes[0];
+    if (rd) {
+      if (0 < L) tb0 = bb[0 + G - 1];
+      if (1 < L) tb1 = bb[1 + G - 1];
+      if (2 < L) tb2 = bb[2 + G - 1];
+      if (3 < L) tb3 = bb[3 + G - 1];
+    }
+  }
+  for (int t0 = 0; t0 < T; t0 += 4) {
+    const uint2 cwc = cw;
+    const uint2 c0 = tb0, c1 = tb1, c2 = tb2, c3 = tb3;
+    if (lead) {
+      const int n0 = t0 + 4;
+      cw = (n0 < L) ? codes[n0 >> 2] : make_uint2(pad4, pad4);
+      if (rd) {
+        tb0 = (n0 + 0 < L) ? bb[n0 + 0 + G - 1] : make_uint2(0, 0);
+        tb1 = (n0 + 1 < L) ? bb[n0 + 1 + G - 1] : make_uint2(0, 0);
+        tb2 = (n0 + 2 < L) ? bb[n0 + 2 + G - 1] : make_uint2(0, 0);
+        tb3 = (n0 + 3 < L) ? bb[n0 + 3 + G - 1] : make_uint2(0, 0);
+      }
+    }
+#pragma unroll
+    for (int j = 0; j < 4; ++j) {
+      uint32_t rH = __shfl_up_sync(FULL, sH, 1, G);
+      uint32_t rF = __shfl_up_sync(FULL, sF, 1, G);
+      uint32_t rC = __shfl_up_sync(FULL, sC, 1, G);
+      if (lead) {
+        const uint32_t w = (j < 2) ? cwc.x : cwc.y;
+        rC = (j & 1) ? (w >> 16) : (w & 0xffffu);
+        const uint2 tv = (j == 0) ? c0 : (j == 1) ? c1 : (j == 2) ? c2 : c3;
+        rH = tv.x;
+        rF = tv.y;
+      }
+      const uint8_t* pa = sprof + (rC & 0xffu) * a.LS + laneoff;
+      const uint8_t* pb = sprof + (rC >> 8) * a.LS + laneoff;
+      gotoh_column<R>(Hl, E, best, hdiag, pa, pb, rH, rF, a.nGe, a.nGsGe);
+      sH = rH;
+      sF = rF;
+      sC = rC;
+      if (wr && tail) bb[t0 + j] = make_uint2(rH, rF);
+    }
+  }
+}
+
+template <int G, int R, int NT>
+__global__ void __launch_bounds__(NT) inter_kernel(InterArgs a) {
+  extern __shared__ __align__(16) uint8_t sprof[];
+  __shared__ int s_chunk;
+  constexpr int NG = NT / G;
+  const int tid = threadIdx.x;
+  const int k = tid & (G - 1);
+  const int g = tid / G;
+  const int npairs = a.pair_end - a.pair_begin;
+  const int nchunks = (npairs + NG - 1) / NG;
+  uint2* __restrict__ bb = a.bbuf + ((size_t)blockIdx.x * NG + g) * (size_t)a.bcap;
+
+  if (a.n_strips == 1) copy_strip(sprof, a.prof, a.SB);
+  for (;;) {
+    if (tid == 0) s_chunk = atomicAdd(a.work_counter, 1);
+    __syncthreads();
+    const int chunk = s_chunk;
+    if (chunk >= nchunks) break;
+    const int p = a.pair_begin + chunk * NG + g;
+    const bool valid = p < a.pair_end;
+    PairRec pr;
+    if (valid) pr = a.pairs[p];
+    else { pr.off = 0; pr.len = 0; pr.id0 = -1; pr.id1 = -1; }
+    int T = pr.len + G;                       // lane G-1 finishes column len-1 at step len+G-2
+    if (G < 32) T = __reduce_max_sync(FULL, T);  // warp-uniform trip count (shuffles)
+    uint32_t best = 0;
+    for (int s = 0; s < a.n_strips; ++s) {
+      if (a.n_strips > 1) {
+        __syncthreads();
+        copy_strip(sprof, a.prof + (size_t)s * a.SB, a.SB);
+        __syncthreads();
+      }
+      strip_pass<G, R>(a, sprof, pr, T, k, s > 0, s + 1 < a.n_strips, bb, best);
+    }
+#pragma unroll
+    for (int o = G / 2; o > 0; o >>= 1) best = __vmaxs2(best, __shfl_xor_sync(FULL, best, o, G));
+    if (valid && k == 0) {
+      const int lo = int(int16_t(best & 0xffffu));
+      const int hi = int(int16_t(best >> 16));
+      a.scores[pr.id0] = lo;
+      if (lo >= a.thr) {
+        const int e = atomicAdd(a.ovf_count, 1);
+        if (e < a.ovf_cap) a.ovf[e] = OvfRec{a.qidx, p, 0, 0};
+      }
+      if (pr.id1 >= 0) {
+        a.scores[pr.id1] = hi;
+        if (hi >= a.thr) {
+          const int e = atomicAdd(a.ovf_count, 1);
+          if (e < a.ovf_cap) a.ovf[e] = OvfRec{a.qidx, p, 1, 0};
+        }
+      }
+    }
+    __syncthreads();
+  }
+}
+
+// ---------------------------------------------------------------------------
+// Instantiation table.
+constexpr int INTER_NT = 256;
+
+#define SW_INTER_CASES(X)                                                          \
+  X(4, 8) X(4, 12) X(4, 16) X(4, 20) X(4, 24) X(4, 28) X(4, 32)                    \
+  X(8, 8) X(8, 12) X(8, 16) X(8, 20) X(8, 24) X(8, 28) X(8, 32)                    \
+  X(16, 8) X(16, 12) X(16, 16) X(16, 20) X(16, 24) X(16, 28) X(16, 32)             \
+  X(32, 8) X(32, 12) X(32, 16) X(32, 20) X(32, 24) X(32, 28) X(32, 32)
+
+typedef void (*inter_fn)(InterArgs);
+
+static inter_fn pick_inter(int G, int R, int NT) {
+  if (NT != INTER_NT) return nullptr;
+#define X(g, r) \
+  if (G == g && R == r) return inter_kernel<g, r, INTER_NT>;
+  SW_INTER_CASES(X)
+#undef X
+  return nullptr;
+}
+
+bool inter_config_supported(int G, int R) { return pick_inter(G, R, INTER_NT) != nullptr; }
+
+int inter_max_ctas_per_sm(int G, int R, int NT, int smem_bytes) {
+  inter_fn f = pick_inter(G, R, NT);
+  if (!f) return 0;
+  if (smem_bytes > 48 * 1024)
+    cudaFuncSetAttribute(f, cudaFuncAttributeMaxDynamicSharedMemorySize, smem_bytes);
+  int n = 0;
+  if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&n, f, NT, smem_bytes) != cudaSuccess) return 0;
+  return n;
+}
+
+cudaError_t launch_inter(int G, int R, int NT, int grid, int smem_bytes, const InterArgs& a, cudaStream_t st) {
+  inter_fn f = pick_inter(G, R, NT);
+  if (!f) return cudaErrorInvalidValue;
+  if (smem_bytes > 48 * 1024) {
+    cudaError_t e = cudaFuncSetAttribute(f, cudaFuncAttributeMaxDynamicSharedMemorySize, smem_bytes);
+    if (e != cudaSuccess) return e;
+  }
+  f<<<grid, NT, smem_bytes, st>>>(a);
+  return cudaGetLastError();
+}
+
+// ---------------------------------------------------------------------------
+// Exact int32 re-score of flagged pairs.  One warp per pair,
+// lane k owns RESCORE_R rows of a 32*RESCORE_R-row strip, same wavefront as the
+// inter-task kernel but one problem per lane and S read from the matrix.
+__global__ void __launch_bounds__(RESCORE_WARPS * 32) rescore_kernel(RescoreArgs a) {
+  constexpr int R = RESCORE_R;
+  constexpr int SW = 33;  // matrix row stride (PAD = alpha <= 32)
+  __shared__ int32_t sm[SW * SW];
+  for (int i = threadIdx.x; i < SW * SW; i += blockDim.x) {
+    const int x = i / SW, y = i % SW;
+    sm[i] = (x < a.alpha && y < a.alpha) ? int(a.matrix[x * a.alpha + y]) : int(PAD_SCORE);
+  }
+  __syncthreads();
+  const int lane = threadIdx.x & 31;
+  const int gw = blockIdx.x * RESCORE_WARPS + threadIdx.x / 32;
+  const int nw = gridDim.x * RESCORE_WARPS;
+  int2* __restrict__ bb = a.bbuf + (size_t)gw * a.bcap;
+  const int cnt = *a.ovf_count;
+  const int pad = a.alpha;
+  for (int e = gw; e < cnt; e += nw) {
+    const OvfRec o = a.ovf[e];
+    const PairRec pr = a.pairs[o.pair];
+    const uint8_t* qc = a.qcodes + a.qoff[o.q];
+    const int m = int(a.qoff[o.q + 1] - a.qoff[o.q]);
+    const int L = pr.len;
+    const int shift = o.half ? 8 : 0;
+    const int nstrips = (m + 32 * R - 1) / (32 * R);
+    int best = 0;
+    for (int s = 0; s < nstrips; ++s) {
+      const bool rd = s > 0, wr = s + 1 < nstrips;
+      int qr[R], Hl[R], E[R];
+#pragma unroll
+      for (int r = 0; r < R; ++r) {
+        const int row = s * 32 * R + lane * R + r;
+        qr[r] = (row < m ? int(qc[row]) : pad) * SW;
+        Hl[r] = 0;
+        E[r] = 0;
+      }
+      int hdiag = 0, sH = 0, sF = 0, sC = pad;
+      const int T = L + 32;
+      for (int t = 0; t < T; ++t) {
+        int rH = __shfl_up_sync(FULL, sH, 1);
+        int rF = __shfl_up_sync(FULL, sF, 1);
+        int rC = __shfl_up_sync(FULL, sC, 1);
+        if (lane == 0) {
+          if (t < L) {
+            rC = (a.stream[pr.off + t] >> shift) & 0xff;
+            if (rd) { const int2 v = bb[t + 31]; rH = v.x; rF = v.y; }
+            else { rH = 0; rF = 0; }
+          } else { rC = pad; rH = 0; rF = 0; }
+        }
+        int hd = hdiag;
+        hdiag = rH;
+        int F = rF;
+#pragma unroll
+        for (int r = 0; r < R; ++r) {
+          const int h = max(max(hd + sm[qr[r] + rC], max(E[r], F)), 0);  // Eq. (2)
+          hd = Hl[r];
+          Hl[r] = h;
+          const int tt = h - a.Gs - a.Ge;
+          E[r] = max(max(E[r] - a.Ge, tt), 0);                            // Eq. (3)
+          F = max(max(F - a.Ge, tt), 0);                                  // Eq. (4)
+          best = max(best, h);
+        }
+        sH = Hl[R - 1];
+        sF = F;
+        sC = rC;
+        if (wr && lane == 31) bb[t] = make_int2(sH, sF);
+      }
+    }
+#pragma unroll
+    for (int off = 16; off > 0; off >>= 1) best = max(best, __shfl_xor_sync(FULL, best, off));
+    if (lane == 0) {
+      const int id = o.half ? pr.id1 : pr.id0;
+      a.scores[(int64_t)o.q * a.n_seqs + id] = best;
+    }
+  }
+}
+
+cudaError_t launch_rescore(int grid, const RescoreArgs& a, cudaStream_t st) {
+  rescore_kernel<<<grid, RESCORE_WARPS * 32, 0, st>>>(a);
+  return cudaGetLastError();
+}
+
+}  // namespace swdual

@@ -1,0 +1,127 @@
+// Host packer: validate, length-sort, pair, interleave.
+//
+// The paper's binary database format gives random access to any sequence and
+// known sizes up front; here the packed form is what the
+// GPU kernels stream:
+//   * non-empty sequences sorted by length, longest first, ties by caller index;
+//   * neighbours paired: pair p = (sorted[2p], sorted[2p+1]); the s16x2 lanes
+//     score both halves of a pair at once, so pairing equal lengths wastes
+//     almost nothing;
+//   * each pair interleaved column by column into 16-bit words
+//     (low byte = id0's residue, high byte = id1's), padded to a multiple of 4
+//     columns with PAD = alphabet_size, 4 columns = one 8-byte load;
+//   * pairs [0, n_long) are longer than t_long (launched separately).
+#include <algorithm>
+#include <atomic>
+#include <stdexcept>
+#include <string>
+#include <thread>
+#include <vector>
+
+#include "../../include/swdual.h"
+#include "sw_internal.h"
+
+namespace swdual {
+
+static unsigned n_threads() { return std::max(1u, std::min(16u, std::thread::hardware_concurrency())); }
+
+void pack_db(const uint8_t* codes, const int64_t* offsets, int64_t n_seqs, int alpha, int64_t t_long, Packed& P) {
+  if (n_seqs < 0) throw std::invalid_argument("n_seqs < 0");
+  if (alpha < 1 || alpha > 32) throw std::invalid_argument("alphabet_size must be in 1..32");
+  if (n_seqs > 0 && !offsets) throw std::invalid_argument("offsets is NULL");
+  if (n_seqs >= (int64_t(1) << 31) - 1) throw std::invalid_argument("more than 2^31-2 sequences");
+  P = Packed{};
+  P.seq_len.resize(size_t(n_seqs));
+  int64_t total = 0;
+  for (int64_t i = 0; i < n_seqs; ++i) {
+    const int64_t L = offsets[i + 1] - offsets[i];
+    if (L < 0) throw std::invalid_argument("offsets not non-decreasing");
+    if (L > (int64_t(1) << 30)) throw std::invalid_argument("sequence longer than 2^30");
+    P.seq_len[size_t(i)] = L;
+    total += L;
+  }
+  if (total > 0 && !codes) throw std::invalid_argument("codes is NULL");
+  P.n_res = total;
+  if (total > 0) {  // every code < alpha (parallel scan)
+    const uint8_t* base = codes + offsets[0];
+    const unsigned nt = n_threads();
+    std::atomic<bool> bad{false};
+    std::vector<std::thread> th;
+    for (unsigned t = 0; t < nt; ++t)
+      th.emplace_back([&, t] {
+        const int64_t a = total * t / nt, b = total * (t + 1) / nt;
+        for (int64_t i = a; i < b; ++i)
+          if (base[i] >= alpha) { bad = true; return; }
+      });
+    for (auto& x : th) x.join();
+    if (bad) throw std::invalid_argument("residue code >= alphabet_size");
+  }
+  std::vector<int32_t> order;
+  order.reserve(size_t(n_seqs));
+  for (int64_t i = 0; i < n_seqs; ++i)
+    if (P.seq_len[size_t(i)] > 0) order.push_back(int32_t(i));
+  std::stable_sort(order.begin(), order.end(),
+                   [&](int32_t a, int32_t b) { return P.seq_len[size_t(a)] > P.seq_len[size_t(b)]; });
+  P.sorted_lens.resize(order.size());
+  for (size_t i = 0; i < order.size(); ++i) P.sorted_lens[i] = P.seq_len[size_t(order[i])];
+  P.max_len = order.empty() ? 0 : P.sorted_lens[0];
+  const size_t np = (order.size() + 1) / 2;
+  P.pairs.resize(np);
+  int64_t off = 0;
+  for (size_t p = 0; p < np; ++p) {
+    PairRec& r = P.pairs[p];
+    r.id0 = order[2 * p];
+    r.id1 = (2 * p + 1 < order.size()) ? order[2 * p + 1] : -1;
+    const int64_t L = P.seq_len[size_t(r.id0)];  // the longer of the two (sorted)
+    r.len = int32_t((L + 3) / 4 * 4);
+    r.off = off;
+    r.pad_ = 0;
+    off += r.len;
+    if (L > t_long) P.n_long = int(p + 1);
+  }
+  P.stream.assign(size_t(std::max<int64_t>(off, 4)), uint16_t(alpha | (alpha << 8)));
+  const uint16_t pad = uint16_t(alpha);
+  const unsigned nt = n_threads();
+  std::vector<std::thread> th;
+  for (unsigned t = 0; t < nt; ++t)
+    th.emplace_back([&, t] {
+      for (size_t p = t; p < np; p += nt) {
+        const PairRec& r = P.pairs[p];
+        const uint8_t* s0 = codes + offsets[r.id0];
+        const int64_t l0 = P.seq_len[size_t(r.id0)];
+        const uint8_t* s1 = r.id1 >= 0 ? codes + offsets[r.id1] : nullptr;
+        const int64_t l1 = r.id1 >= 0 ? P.seq_len[size_t(r.id1)] : 0;
+        uint16_t* w = P.stream.data() + r.off;
+        for (int64_t c = 0; c < r.len; ++c) {
+          const uint16_t a = c < l0 ? s0[c] : pad;
+          const uint16_t b = c < l1 ? s1[c] : pad;
+          w[c] = uint16_t(a | (b << 8));
+        }
+      }
+    });
+  for (auto& x : th) x.join();
+}
+
+}  // namespace swdual
+
+// Host-only access to the packer (tests, tooling): two-phase, call with
+// pairs == NULL / stream == NULL to get the sizes first.
+extern "C" int32_t sw_pack_db_host(const uint8_t* codes, const int64_t* offsets, int64_t n_seqs, int32_t alphabet_size,
+                                   int64_t t_long, sw_pair_t* pairs, int64_t* n_pairs, uint16_t* stream,
+                                   int64_t* stream_words, int64_t* n_long) {
+  static_assert(sizeof(sw_pair_t) == sizeof(swdual::PairRec), "sw_pair_t layout");
+  try {
+    swdual::Packed P;
+    swdual::pack_db(codes, offsets, n_seqs, alphabet_size, t_long, P);
+    if (n_pairs) *n_pairs = int64_t(P.pairs.size());
+    if (stream_words) *stream_words = int64_t(P.stream.size());
+    if (n_long) *n_long = P.n_long;
+    if (pairs) std::copy(P.pairs.begin(), P.pairs.end(), reinterpret_cast<swdual::PairRec*>(pairs));
+    if (stream) std::copy(P.stream.begin(), P.stream.end(), stream);
+    return SW_OK;
+  } catch (const std::invalid_argument&) {
+    return SW_EINVAL;
+  } catch (...) {
+    return SW_ENOMEM;
+  }
+}

@@ -1,0 +1,92 @@
+// Device-side building blocks of the Gotoh cell update on sm_100a DPX.
+//
+// Recurrences (sec. II.B, Eqs. (2)-(4), L178-194), s = query (rows i),
+// t = database sequence (columns j):
+//   H_ij = max(H_{i-1,j-1} + S_ij, E_ij, F_ij, 0)
+//   E_ij = -Ge + max(E_{i,j-1}, H_{i,j-1} - Gs)
+//   F_ij = -Ge + max(F_{i-1,j}, H_{i-1,j} - Gs)
+// E and F are clamped at 0 (exact: H >= 0 absorbs any negative E/F, DESIGN.md
+// reading R-9), so every stored value lies in [0, 32767] and the H maximum
+// detects the only possible (upward) int16 wrap.
+//
+// Two independent problems share every 32-bit register (s16x2): the low half
+// scores the query against DB sequence id0 of a pair, the high half against id1.
+// Per cell pair: VIMNMX (max E,F) + VIADDMNMX (H) + VIADD.16x2 (H-Gs-Ge) +
+// 2x VIADDMNMX.RELU (E', F') + 1/2 VIMNMX3 (running max) = 5.5 DPX lane-ops,
+// plus one sign-extending PRMT that builds the (S[q_i][a], S[q_i][b]) word from
+// the int8 query profile rows of the two DB letters a, b.
+#pragma once
+#include <cstdint>
+
+namespace swdual {
+
+__device__ __forceinline__ uint32_t prmt(uint32_t a, uint32_t b, uint32_t sel) {
+  uint32_t d;
+  asm("prmt.b32 %0, %1, %2, %3;" : "=r"(d) : "r"(a), "r"(b), "r"(sel));
+  return d;
+}
+
+// Selector that turns int8 row j (0..3) of word a (letter of id0) and word b
+// (letter of id1) into the s16x2 word (sext a_j, sext b_j): the msb of a PRMT
+// selector nibble replicates the sign of the selected byte.
+__host__ __device__ constexpr uint32_t pair_sel(int j) {
+  return uint32_t(j) | (uint32_t(j | 8) << 4) | (uint32_t(4 + j) << 8) | (uint32_t((4 + j) | 8) << 12);
+}
+
+template <int R>
+struct ProfUnit {
+  static constexpr int BYTES = (R % 8 == 0) ? 8 : 4;  // LDS.64 or LDS.32 per letter
+};
+
+// Lane block size in bytes for R int8 rows: an odd number of load units so that
+// consecutive lanes of a group hit distinct shared-memory banks.
+__host__ __device__ constexpr int lane_block_bytes(int R) {
+  return ((R % 8 == 0) ? (((R / 8) | 1) * 8) : (((R / 4) | 1) * 4));
+}
+
+// One column of R rows for one lane.
+//   Hl[r]  : in H_{r,j-1}, out H_{r,j}
+//   E[r]   : in E_{r,j},   out E_{r,j+1}
+//   hdiag  : in H_{top-1, j-1}, out H_{top-1, j}  (top boundary of the previous column)
+//   Hio    : in H_{top-1, j} (from the lane above), out H_{bottom, j}
+//   Fio    : in F_{top, j},                        out F_{bottom+1, j}
+template <int R>
+__device__ __forceinline__ void gotoh_column(uint32_t (&Hl)[R], uint32_t (&E)[R], uint32_t& best,
+                                             uint32_t& hdiag, const uint8_t* __restrict__ pa,
+                                             const uint8_t* __restrict__ pb, uint32_t& Hio, uint32_t& Fio,
+                                             uint32_t nGe, uint32_t nGsGe) {
+  uint32_t hd = hdiag;
+  hdiag = Hio;
+  uint32_t F = Fio;
+  uint32_t hprev = 0;
+  constexpr int UB = ProfUnit<R>::BYTES;
+#pragma unroll
+  for (int u = 0; u < R / UB; ++u) {
+    uint32_t wa[UB / 4], wb[UB / 4];
+    if constexpr (UB == 8) {
+      const uint2 x = *reinterpret_cast<const uint2*>(pa + u * 8);
+      const uint2 y = *reinterpret_cast<const uint2*>(pb + u * 8);
+      wa[0] = x.x; wa[1] = x.y; wb[0] = y.x; wb[1] = y.y;
+    } else {
+      wa[0] = *reinterpret_cast<const uint32_t*>(pa + u * 4);
+      wb[0] = *reinterpret_cast<const uint32_t*>(pb + u * 4);
+    }
+#pragma unroll
+    for (int j = 0; j < UB; ++j) {
+      const int r = u * UB + j;
+      const uint32_t s = prmt(wa[j >> 2], wb[j >> 2], pair_sel(j & 3));
+      const uint32_t h = __viaddmax_s16x2(hd, s, __vmaxs2(E[r], F));   // Eq. (2)
+      hd = Hl[r];
+      Hl[r] = h;
+      const uint32_t t = __vadd2(h, nGsGe);                              // H - Gs - Ge
+      E[r] = __viaddmax_s16x2_relu(E[r], nGe, t);                        // Eq. (3)
+      F = __viaddmax_s16x2_relu(F, nGe, t);                              // Eq. (4)
+      if (r & 1) best = __vimax3_s16x2(best, hprev, h);
+      else hprev = h;
+    }
+  }
+  Hio = Hl[R - 1];
+  Fio = F;
+}
+
+}  // namespace swdual

@@ -1,0 +1,96 @@
+// Internal types shared by the host engine (engine.cpp) and the kernels (kernels.cu).
+// Product code only: nothing here is shared with oracle/.
+#pragma once
+#include <cstdint>
+#include <vector>
+#include <cuda_runtime.h>
+
+namespace swdual {
+
+// One packed database "pair": two length-sorted neighbours interleaved column by
+// column into 16-bit words (low byte = sequence id0, high byte = id1), padded to a
+// multiple of 4 columns with the PAD code.  id1 = -1 for an odd leftover sequence.
+struct PairRec {
+  int64_t off;   // start, in 16-bit words, into the pair stream (multiple of 4)
+  int32_t len;   // padded length (multiple of 4) = columns processed
+  int32_t id0;   // caller's index of the low-half sequence
+  int32_t id1;   // caller's index of the high-half sequence or -1
+  int32_t pad_;
+};
+
+// Host-packed database (packer.cpp).
+struct Packed {
+  std::vector<PairRec> pairs;        // sorted longest first
+  std::vector<uint16_t> stream;      // interleaved pair columns
+  std::vector<int64_t> seq_len;      // caller order
+  std::vector<int64_t> sorted_lens;  // non-empty lengths, descending
+  int64_t n_res = 0, max_len = 0;
+  int n_long = 0;                    // pairs [0, n_long) are longer than t_long
+};
+void pack_db(const uint8_t* codes, const int64_t* offsets, int64_t n_seqs, int alpha, int64_t t_long, Packed& P);
+
+// A pair whose int16 maximum reached the overflow threshold:
+// re-scored exactly in int32.
+struct OvfRec {
+  int32_t q;     // query index within the search
+  int32_t pair;  // pair index
+  int32_t half;  // 0 = id0, 1 = id1
+  int32_t pad_;
+};
+
+// Geometry of one query profile (int8, strip-major, lane-blocked; see kernels.cu).
+struct ProfGeom {
+  int G, R;        // lanes per group, rows per lane
+  int LB;          // bytes per lane block (>= R, odd number of load units)
+  int LS;          // bytes per letter = G * LB
+  int NL;          // letters = alpha + 1 (PAD = alpha)
+  int SB;          // bytes per strip (multiple of 16)
+  int n_strips;    // ceil(m / (G*R))
+};
+
+struct InterArgs {
+  const uint8_t* prof;       // [n_strips][SB]
+  int n_strips, SB, LS, LB;
+  const uint16_t* stream;
+  const PairRec* pairs;
+  int pair_begin, pair_end;  // [begin, end) pairs of this launch
+  uint2* bbuf;               // boundary rows, [gridDim][NG][bcap]
+  int bcap;
+  int* work_counter;
+  int32_t* scores;           // row of this query: scores[id]
+  int32_t thr;               // overflow threshold (int16 max >= thr -> re-score)
+  OvfRec* ovf;
+  int* ovf_count;
+  int ovf_cap;
+  int qidx;
+  uint32_t code_pad2;        // PAD | PAD << 8
+  uint32_t nGe, nGsGe;       // packed s16x2 -Ge, -(Gs+Ge)
+};
+
+struct RescoreArgs {
+  const uint8_t* qcodes;     // all queries, concatenated
+  const int64_t* qoff;       // [nq+1]
+  const uint16_t* stream;
+  const PairRec* pairs;
+  const int8_t* matrix;      // alpha x alpha
+  int alpha;
+  const OvfRec* ovf;
+  const int* ovf_count;
+  int2* bbuf;                // [gridDim*warps][bcap]
+  int bcap;
+  int32_t* scores;           // [nq][n_seqs]
+  int64_t n_seqs;
+  int32_t Gs, Ge;
+};
+
+// kernels.cu entry points (host side launchers); return cudaError_t
+cudaError_t launch_build_profile(const uint8_t* q, int m, const int8_t* matrix, int alpha,
+                                 const ProfGeom& g, uint8_t* prof, cudaStream_t st);
+int inter_max_ctas_per_sm(int G, int R, int NT, int smem_bytes);
+cudaError_t launch_inter(int G, int R, int NT, int grid, int smem_bytes, const InterArgs& a, cudaStream_t st);
+bool inter_config_supported(int G, int R);
+cudaError_t launch_rescore(int grid, const RescoreArgs& a, cudaStream_t st);
+constexpr int RESCORE_WARPS = 4;
+constexpr int RESCORE_R = 8;
+
+}  // namespace swdual

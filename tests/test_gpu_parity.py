@@ -1,0 +1,191 @@
+"""GPU parity: the CUDA path (through the C ABI) vs the CPU oracle, bit-exact.
+
+Inputs are seeded and synthetic (swgen).  Sizes span several strips, lane
+groups and chunks with ragged tails; edge cases cover empty sequences, length
+1..5, strip boundaries, every kernel geometry, forced and real int16 overflow.
+"""
+import numpy as np
+import pytest
+
+import oracle
+import swgen
+from oracle.blosum62 import blosum62 as oracle_b62
+
+pytestmark = pytest.mark.gpu
+
+B62_ORACLE = oracle_b62()
+
+
+def _pkg():
+    import paper_conf_icpp_kedad_sidhoummmmt14_b200 as sw
+    return sw
+
+
+def gpu_scores(qc, qo, dc, do, S=None, gs=10, ge=2, alpha=24, opts=None, device_out=False):
+    sw = _pkg()
+    S = sw.blosum62() if S is None else S
+    with sw.Handle(0) as h:
+        for k, v in (opts or {}).items():
+            h.set_option(k, v)
+        db = h.load_db(dc, do, alphabet_size=alpha)
+        if device_out:
+            import torch
+            out = h.search(qc, qo, db, S, gs, ge)
+            torch.cuda.synchronize()
+            return out.cpu().numpy()
+        out = np.zeros((len(qo) - 1, len(do) - 1), dtype=np.int32)
+        return h.search(qc, qo, db, S, gs, ge, out=out)
+
+
+def oracle_scores(qc, qo, dc, do, S=None, gs=10, ge=2, procs=8):
+    S = B62_ORACLE if S is None else S
+    return oracle.gotoh_search(qc, qo, dc, do, S, gs, ge, procs=procs)
+
+
+def _seqs(lengths, rng, alpha=20):
+    lens = np.asarray(lengths, dtype=np.int64)
+    off = np.zeros(len(lens) + 1, dtype=np.int64)
+    np.cumsum(lens, out=off[1:])
+    return rng.integers(0, alpha, size=int(off[-1])).astype(np.uint8), off
+
+
+def test_matrix_tables_agree():
+    sw = _pkg()
+    np.testing.assert_array_equal(sw.blosum62().astype(np.int32), B62_ORACLE)
+
+
+def test_small_random_edges():
+    rng = np.random.default_rng(11)
+    dl = [0, 1, 2, 3, 4, 5, 7, 8, 31, 32, 33, 63, 64, 65, 127, 128, 129, 255, 256, 257, 300, 511, 512, 513, 0]
+    dl += list(rng.integers(1, 700, size=300))
+    dc, do = _seqs(dl, rng, alpha=24)
+    ql = [1, 2, 7, 8, 9, 31, 32, 33, 64, 100, 255, 256, 257, 500, 767, 768, 769, 1025]
+    qc, qo = _seqs(ql, rng, alpha=24)
+    np.testing.assert_array_equal(gpu_scores(qc, qo, dc, do), oracle_scores(qc, qo, dc, do))
+
+
+@pytest.mark.parametrize("G", [4, 8, 16, 32])
+@pytest.mark.parametrize("R", [8, 12, 16, 20, 24, 28, 32])
+def test_every_geometry(G, R):
+    rng = np.random.default_rng(1000 + 37 * G + R)
+    dl = list(rng.integers(1, 300, size=90)) + [0, 1, 3, 5]
+    dc, do = _seqs(dl, rng)
+    # one query spanning 1 strip exactly, one ragged multi-strip
+    ql = [G * R, 2 * G * R + 3, 5]
+    qc, qo = _seqs(ql, rng)
+    got = gpu_scores(qc, qo, dc, do, opts={"force_G": G, "force_R": R})
+    np.testing.assert_array_equal(got, oracle_scores(qc, qo, dc, do))
+
+
+def test_config_c1_full():
+    c = swgen.make_config("c1")
+    got = gpu_scores(c["qcodes"], c["qoff"], c["dcodes"], c["doff"])
+    ref = oracle_scores(c["qcodes"], c["qoff"], c["dcodes"], c["doff"])
+    np.testing.assert_array_equal(got, ref)
+    assert got.max() > 300  # planted homologs score high
+
+
+def test_device_output_and_gap_params():
+    rng = np.random.default_rng(12)
+    dc, do = _seqs(rng.integers(1, 400, size=200), rng)
+    qc, qo = _seqs([150, 333], rng)
+    for gs, ge in ((10, 2), (0, 1), (11, 1), (5, 5), (0, 0)):
+        got = gpu_scores(qc, qo, dc, do, gs=gs, ge=ge, device_out=True)
+        np.testing.assert_array_equal(got, oracle_scores(qc, qo, dc, do, gs=gs, ge=ge))
+
+
+def test_asymmetric_matrix_small_alphabet():
+    rng = np.random.default_rng(13)
+    A = 5
+    S = rng.integers(-5, 9, size=(A, A)).astype(np.int8)
+    dc, do = _seqs(rng.integers(1, 200, size=150), rng, alpha=A)
+    qc, qo = _seqs([77, 260], rng, alpha=A)
+    got = gpu_scores(qc, qo, dc, do, S=S, gs=3, ge=1, alpha=A)
+    np.testing.assert_array_equal(got, oracle_scores(qc, qo, dc, do, S=S.astype(np.int32), gs=3, ge=1))
+
+
+def test_forced_overflow_rescore():
+    """A tiny threshold sends most pairs through the int32 re-score path."""
+    rng = np.random.default_rng(14)
+    dc, do = _seqs(rng.integers(1, 500, size=120), rng)
+    qc, qo = _seqs([200, 900], rng)
+    sw = _pkg()
+    with sw.Handle(0) as h:
+        h.set_option("overflow_threshold", 40)
+        db = h.load_db(dc, do)
+        out = np.zeros((2, 120), dtype=np.int32)
+        h.search(qc, qo, db, sw.blosum62(), 10, 2, out=out)
+        st = h.last_stats()
+    np.testing.assert_array_equal(out, oracle_scores(qc, qo, dc, do))
+    assert st["n_overflow"] > 0
+
+
+def test_real_int16_overflow():
+    """Self-hits of W-rich sequences longer than 32767/11 really wrap int16."""
+    rng = np.random.default_rng(15)
+    W = 17  # 'W' in NCBI order
+    q = np.full(3200, W, dtype=np.uint8)
+    q[rng.integers(0, 3200, 40)] = rng.integers(0, 20, 40)
+    mut = q.copy()
+    mut[rng.integers(0, 3200, 100)] = rng.integers(0, 20, 100)
+    dl_other = list(rng.integers(1, 300, size=50))
+    others, oo = _seqs(dl_other, rng)
+    parts = [q, mut, others]
+    dc = np.concatenate(parts)
+    do = np.concatenate([[0, len(q), len(q) + len(mut)], len(q) + len(mut) + oo[1:]]).astype(np.int64)
+    qc, qo = q.copy(), np.array([0, len(q)], dtype=np.int64)
+    got = gpu_scores(qc, qo, dc, do)
+    ref = oracle_scores(qc, qo, dc, do)
+    assert ref.max() > 32767
+    np.testing.assert_array_equal(got, ref)
+
+
+def test_empty_cases():
+    sw = _pkg()
+    rng = np.random.default_rng(16)
+    dc, do = _seqs([0, 0, 0], rng)
+    qc, qo = _seqs([10, 0], rng)
+    np.testing.assert_array_equal(gpu_scores(qc, qo, dc, do), np.zeros((2, 3), np.int32))
+    dc, do = _seqs([5, 9], rng)
+    qc, qo = _seqs([], rng)
+    assert gpu_scores(qc, qo, dc, do).shape == (0, 2)
+
+
+def test_errors():
+    sw = _pkg()
+    rng = np.random.default_rng(17)
+    dc, do = _seqs([5, 9], rng)
+    with sw.Handle(0) as h:
+        bad = dc.copy()
+        bad[0] = 24
+        with pytest.raises(sw.SWError):
+            h.load_db(bad, do, alphabet_size=24)
+        with pytest.raises(sw.SWError):
+            h.load_db(dc, do, alphabet_size=33)
+        db = h.load_db(dc, do)
+        qc, qo = _seqs([4], rng)
+        out = np.zeros((1, 2), np.int32)
+        with pytest.raises(sw.SWError):
+            h.search(qc, qo, db, sw.blosum62(), -1, 2, out=out)
+        with pytest.raises(sw.SWError):
+            h.search(np.array([30, 1, 2, 3], np.uint8), qo, db, sw.blosum62(), 10, 2, out=out)
+
+
+@pytest.mark.parametrize("name", ["c2", "c3"])
+def test_swissprot_scale_sampled(name):
+    """BASELINE configs 2/3 at full size on the GPU; the oracle checks a seeded
+    sample of DB sequences (plus every planted homolog and the top hits)."""
+    c = swgen.make_config(name)
+    got = gpu_scores(c["qcodes"], c["qoff"], c["dcodes"], c["doff"])
+    N = len(c["doff"]) - 1
+    rng = np.random.default_rng(99)
+    sample = set(rng.choice(N, size=300 if name == "c3" else 2000, replace=False).tolist())
+    sample |= {p[0] for p in c["plants"]}
+    sample |= set(np.argsort(got.max(axis=0))[-20:].tolist())
+    idx = np.array(sorted(sample), dtype=np.int64)
+    lens = c["doff"][idx + 1] - c["doff"][idx]
+    sub_off = np.zeros(len(idx) + 1, dtype=np.int64)
+    np.cumsum(lens, out=sub_off[1:])
+    sub = np.concatenate([c["dcodes"][c["doff"][i]:c["doff"][i + 1]] for i in idx])
+    ref = oracle_scores(c["qcodes"], c["qoff"], sub, sub_off, procs=16)
+    np.testing.assert_array_equal(got[:, idx], ref)

@@ -1,0 +1,380 @@
+#!/usr/bin/env python
+"""bench.py -- whole-box GCUPS of the SWDUAL hot path on B200 (BASELINE.json metric).
+
+One step = one pass of the whole hot path over the workload: every (query,
+shard) task scored by sw_search on its GPU (profile build, inter-task DPX
+kernels, int32 re-score) plus the single collective, the all-gather of the
+int32 score blocks (N > 1).  Workload (default): BASELINE config 3, the 20-query
+sweep (144..5478 aa) against the Swiss-Prot-sized synthetic DB (570k seqs,
+205M residues) -- the configuration the metric "GCUPS at 1/2/4/8 B200" is
+quoted on; the DB is cut into N shards and placed by the dual approximation.
+
+  python bench.py [--gpus N] [--steps K] [--warmup W] [--impl ours|reference]
+  torchrun --nproc-per-node N bench.py --gpus N ...
+
+Rank 0 prints ONE JSON line.  GCUPS = sum_q m_q * sum_d n_d / t / 1e9 (real
+residues), t = max over ranks of the CUDA-event time of the
+K timed steps.  --impl reference times the CPU oracle (the only reference this
+paper-only tier has) on a bounded sample of the same workload.
+"""
+from __future__ import annotations
+
+import argparse
+import json
+import os
+import statistics
+import subprocess
+import sys
+import threading
+import time
+
+import numpy as np
+
+ROOT = os.path.dirname(os.path.abspath(__file__))
+sys.path.insert(0, ROOT)
+
+import swgen  # noqa: E402
+
+METRIC = "GCUPS (whole box, device-timed) at 1/2/4/8 B200; fraction of DPX cell roofline"
+WORKLOADS = {
+    "c3": "BASELINE config 3: 20-query sweep 144-5478 aa vs Swiss-Prot-sized synthetic DB (570k seqs, ~205M residues), BLOSUM62, gap 10/2",
+    "c2": "BASELINE config 2: 1 query (567 aa) vs Swiss-Prot-sized synthetic DB (570k seqs, ~205M residues), BLOSUM62, gap 10/2",
+    "c1": "BASELINE config 1: 1 query (144 aa) vs 1,000 synthetic sequences, BLOSUM62, gap 10/2",
+    "c4": "BASELINE config 4: queries 2,000-35,000 aa vs 1,500 long synthetic sequences (>3,000 aa)",
+}
+REASONS = {0x1: "gpu_idle", 0x2: "applications_clocks_setting", 0x4: "sw_power_cap", 0x8: "hw_slowdown",
+           0x10: "sync_boost", 0x20: "sw_thermal_slowdown", 0x40: "hw_thermal_slowdown",
+           0x80: "hw_power_brake_slowdown", 0x100: "display_clock_setting"}
+# DPX ALU pipe: 64 lanes/clk/SM (16 per SMSP, measured by tools/dpx_microbench.cu: 18.4 T lane-ops/s);
+# the Gotoh s16x2 update needs 5.5 lane-ops per 2 cells.
+ALU_LANES_PER_SM_CLK = 64
+OPS_PER_CELL = 2.75
+
+
+def parse():
+    ap = argparse.ArgumentParser()
+    ap.add_argument("--gpus", type=int, default=1)
+    ap.add_argument("--steps", type=int, default=5)
+    ap.add_argument("--warmup", type=int, default=3)
+    ap.add_argument("--impl", default="ours", choices=["ours", "reference"])
+    ap.add_argument("--workload", default="c3", choices=sorted(WORKLOADS))
+    ap.add_argument("--n-db", type=int, default=None, help="override DB size (smoke runs only)")
+    ap.add_argument("--e2e-steps", type=int, default=2)
+    ap.add_argument("--no-cpu-baseline", action="store_true")
+    ap.add_argument("--cpu-baseline-cells", type=float, default=3.0e10)
+    return ap.parse_args()
+
+
+class ClockSampler:
+    """nvidia-smi clocks + throttle reasons sampled every 200 ms during the timed region."""
+
+    def __init__(self, dev: int):
+        self.dev = dev
+        self.lines: list[str] = []
+        self.proc = None
+        self.th = None
+
+    def start(self):
+        try:
+            self.proc = subprocess.Popen(
+                ["nvidia-smi", "-i", str(self.dev), "--query-gpu=clocks.sm,clocks.max.sm,clocks_event_reasons.active,power.draw",
+                 "--format=csv,noheader,nounits", "-lms", "200"],
+                stdout=subprocess.PIPE, stderr=subprocess.DEVNULL, text=True)
+        except Exception:
+            self.proc = None
+            return
+        self.th = threading.Thread(target=self._read, daemon=True)
+        self.th.start()
+
+    def _read(self):
+        for line in self.proc.stdout:
+            self.lines.append(line.strip())
+
+    def stop(self) -> dict:
+        if self.proc is None:
+            return {"sm_mhz": None, "sm_max_mhz": None, "reasons": ["nvidia-smi unavailable"]}
+        time.sleep(0.25)
+        self.proc.terminate()
+        try:
+            self.proc.wait(timeout=5)
+        except Exception:
+            self.proc.kill()
+        if self.th:
+            self.th.join(timeout=2)
+        sm, smax, reasons, power = [], [], set(), []
+        for ln in self.lines:
+            parts = [p.strip() for p in ln.split(",")]
+            if len(parts) < 3:
+                continue
+            try:
+                sm.append(float(parts[0]))
+                smax.append(float(parts[1]))
+                bits = int(parts[2], 16)
+                power.append(float(parts[3]) if len(parts) > 3 else 0.0)
+            except ValueError:
+                continue
+            for b, name in REASONS.items():
+                if bits & b and name != "gpu_idle":
+                    reasons.add(name)
+        load = [x for x in sm if x > 500] or sm
+        return {"sm_mhz": statistics.median(load) if load else None,
+                "sm_max_mhz": max(smax) if smax else None,
+                "reasons": sorted(reasons), "samples": len(sm),
+                "power_w_max": max(power) if power else None}
+
+
+def workload(args):
+    c = swgen.make_config(args.workload, n_db=args.n_db)
+    q_lens = np.diff(c["qoff"]).astype(np.int64)
+    d_lens = np.diff(c["doff"]).astype(np.int64)
+    return c, q_lens, d_lens
+
+
+def config_obj(args, c, q_lens, d_lens, n):
+    return {"workload": WORKLOADS[args.workload], "name": args.workload,
+            "n_queries": int(len(q_lens)), "query_residues": int(q_lens.sum()),
+            "n_db_seqs": int(len(d_lens)), "db_residues": int(d_lens.sum()),
+            "matrix": "BLOSUM62", "gap_open": 10, "gap_extend": 2,
+            "shards": n, "placement": "dual-approximation (query, shard) tasks",
+            "l2": "inputs larger than L2: 205 MB packed DB > 126 MB L2, streamed once per query per step"
+            if args.workload in ("c2", "c3") and args.n_db is None else "small workload"}
+
+
+def cpu_baseline(c, target_cells: float, seed: int = 2024) -> dict:
+    """The oracle as it stands, on a bounded random sample of the workload's DB, all host cores."""
+    import oracle
+    from oracle.blosum62 import blosum62 as ob62
+    d_lens = np.diff(c["doff"])
+    qsum = int(np.diff(c["qoff"]).sum())
+    rng = np.random.default_rng(seed)
+    n = len(d_lens)
+    want_res = max(1.0, target_cells / max(qsum, 1))
+    k = int(min(n, max(1, want_res / max(d_lens.mean(), 1))))
+    idx = np.sort(rng.choice(n, size=k, replace=False))
+    lens = d_lens[idx]
+    off = np.zeros(k + 1, dtype=np.int64)
+    np.cumsum(lens, out=off[1:])
+    sub = np.concatenate([c["dcodes"][c["doff"][i]:c["doff"][i + 1]] for i in idx]) if k else np.zeros(0, np.uint8)
+    cores = os.cpu_count() or 1
+    oracle.build()
+    t0 = time.perf_counter()
+    oracle.gotoh_search(c["qcodes"], c["qoff"], sub, off, ob62(), 10, 2, procs=cores)
+    dt = time.perf_counter() - t0
+    cells = float(qsum) * float(lens.sum())
+    return {"value": round(cells / dt / 1e9, 4), "unit": "GCUPS", "cores": cores, "kind": "oracle",
+            "sample": f"{k} seeded-random DB sequences ({int(lens.sum())} residues) x all {len(c['qoff']) - 1} queries "
+                      f"= {cells:.3e} cells in {dt:.1f} s"}
+
+
+def run_reference(args):
+    rank = int(os.environ.get("RANK", "0"))
+    if rank != 0:
+        return
+    c, q_lens, d_lens = workload(args)
+    import oracle
+    from oracle.blosum62 import blosum62 as ob62
+    oracle.build()
+    cores = os.cpu_count() or 1
+    qsum = int(q_lens.sum())
+    per_step_cells = 5.0e9
+    k = int(max(1, min(len(d_lens), per_step_cells / qsum / max(d_lens.mean(), 1))))
+    rng = np.random.default_rng(7)
+    times, cells_done = [], []
+    for step in range(args.warmup + args.steps):
+        idx = np.sort(rng.choice(len(d_lens), size=k, replace=False))
+        lens = d_lens[idx]
+        off = np.zeros(k + 1, dtype=np.int64)
+        np.cumsum(lens, out=off[1:])
+        sub = np.concatenate([c["dcodes"][c["doff"][i]:c["doff"][i + 1]] for i in idx])
+        t0 = time.perf_counter()
+        oracle.gotoh_search(c["qcodes"], c["qoff"], sub, off, ob62(), 10, 2, procs=cores)
+        dt = time.perf_counter() - t0
+        if step >= args.warmup:
+            times.append(dt)
+            cells_done.append(float(qsum) * float(lens.sum()))
+    T = sum(times)
+    value = sum(cells_done) / T / 1e9
+    line = {"metric": METRIC, "value": round(value, 4), "unit": "GCUPS", "n_gpus": args.gpus, "steps": args.steps,
+            "warmup": args.warmup, "ms_per_step": round(1e3 * T / args.steps, 3), "higher_is_better": True,
+            "scaling": "strong", "vs_baseline": None, "dtype": "int32", "data": "synthetic",
+            "config": config_obj(args, c, q_lens, d_lens, 1), "impl": "reference",
+            "cpu_baseline": {"value": round(value, 4), "unit": "GCUPS", "cores": cores, "kind": "oracle",
+                             "sample": f"per step {k} seeded-random DB sequences x all queries (~{per_step_cells:.1e} cells)"},
+            "e2e": {"value": round(value, 4), "unit": "GCUPS", "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0}}
+    print(json.dumps(line), flush=True)
+
+
+def run_ours(args):
+    import torch
+    import paper_conf_icpp_kedad_sidhoummmmt14_b200 as sw
+    from paper_conf_icpp_kedad_sidhoummmmt14_b200 import dist as swdist
+
+    rank = int(os.environ.get("RANK", "0"))
+    world = int(os.environ.get("WORLD_SIZE", "1"))
+    local = int(os.environ.get("LOCAL_RANK", "0"))
+    if world != args.gpus:
+        if world == 1 and args.gpus > 1:
+            raise SystemExit("--gpus N > 1 needs torchrun --nproc-per-node N")
+    torch.cuda.set_device(local)
+    dev = torch.device("cuda", local)
+    pg = None
+    if world > 1:
+        import torch.distributed as tdist
+        tdist.init_process_group("nccl", device_id=dev)
+        pg = tdist
+
+    def barrier():
+        if pg is not None:
+            pg.barrier()
+
+    c, q_lens, d_lens = workload(args)
+    Q, N = len(q_lens), len(d_lens)
+    total_cells = float(q_lens.sum()) * float(d_lens.sum())
+    shards = swdist.shard_cut(c["doff"], world)
+    shard_res = [int(d_lens[s].sum()) for s in shards]
+    plan = swdist.place(q_lens, shards, shard_res, world)
+    blocks = swdist.local_blocks(plan, rank)
+
+    S = sw.blosum62()
+    h = sw.Handle(local, timing=True)
+    dbs = {}
+    for s, _qs in blocks:
+        sc, so = swdist.subset(c["dcodes"], c["doff"], shards[s])
+        dbs[s] = h.load_db(sc, so, alphabet_size=24)
+    # per block: query subset (host), device output view into one flat buffer
+    sizes = [swdist.flat_size(plan, r) for r in range(world)]
+    cap = max(max(sizes), 1)
+    flat = torch.zeros(cap, dtype=torch.int32, device=dev)
+    gathered = torch.empty(world * cap, dtype=torch.int32, device=dev) if world > 1 else None
+    jobs = []
+    pos = 0
+    for s, qs in blocks:
+        qc, qo = swdist.subset(c["qcodes"], c["qoff"], qs)
+        n = len(shards[s])
+        view = flat[pos:pos + len(qs) * n].view(len(qs), n)
+        pos += len(qs) * n
+        jobs.append((s, qs, qc, qo, view))
+    stream = torch.cuda.current_stream(dev)
+
+    def step():
+        for s, qs, qc, qo, view in jobs:
+            h.search(qc, qo, dbs[s], S, 10, 2, out=view, stream=stream)
+        if world > 1:
+            pg.all_gather_into_tensor(gathered, flat)
+
+    for _ in range(args.warmup):
+        step()
+    torch.cuda.synchronize()
+    h.set_option("timing_accumulate", 1)
+    h.set_option("timing_reset", 1)
+    clocks = ClockSampler(local)
+    clocks.start()
+    barrier()
+    torch.cuda.synchronize()
+    e0 = torch.cuda.Event(enable_timing=True)
+    e1 = torch.cuda.Event(enable_timing=True)
+    e0.record(stream)
+    for _ in range(args.steps):
+        step()
+    e1.record(stream)
+    torch.cuda.synchronize()
+    barrier()
+    clk = clocks.stop()
+    ms_local = e0.elapsed_time(e1)
+    st = h.last_stats()
+    ms = torch.tensor([ms_local], dtype=torch.float64, device=dev)
+    if pg is not None:
+        pg.all_reduce(ms, op=pg.ReduceOp.MAX)
+    T = float(ms.item())
+    value = total_cells * args.steps / (T / 1e3) / 1e9
+
+    # dominant kernel: inter-task kernel over the short pairs (>= 95% of cells); the
+    # library's own accounting of one step gives its cells and the launch count
+    h.set_option("timing_accumulate", 0)
+    cells_short_step = 0.0
+    n_launch_step = 0
+    for s, qs, qc, qo, view in jobs:
+        h.search(qc, qo, dbs[s], S, 10, 2, out=view, stream=stream)
+        one = h.last_stats()
+        cells_short_step += one["cells_short"]
+        n_launch_step += one["n_launches"]
+    torch.cuda.synchronize()
+    sm_max = clk.get("sm_max_mhz") or 1965.0
+    n_sm = torch.cuda.get_device_properties(dev).multi_processor_count
+    peak = n_sm * ALU_LANES_PER_SM_CLK * sm_max * 1e6 / OPS_PER_CELL / 1e9
+    achieved = cells_short_step * args.steps / (st["short_ms"] / 1e3) / 1e9 if st["short_ms"] > 0 else None
+    traffic = None
+    tpath = os.path.join(ROOT, "profiles", "traffic.json")
+    if os.path.exists(tpath):
+        try:
+            traffic = json.load(open(tpath)).get(args.workload)
+        except Exception:
+            traffic = None
+
+    # e2e through the public API with host buffers
+    e2e = None
+    if args.e2e_steps > 0:
+        host_out = {}
+        for s, qs, qc, qo, view in jobs:
+            host_out[s] = torch.empty(tuple(view.shape), dtype=torch.int32, pin_memory=True).numpy()
+        final_host = torch.empty(world * cap, dtype=torch.int32, pin_memory=True) if world > 1 else None
+        h2d = sum(int(qc.nbytes + qo.nbytes + S.nbytes) for _s, _q, qc, qo, _v in jobs)
+        d2h = sum(int(v.numel() * 4) for *_x, v in jobs) if world == 1 else world * cap * 4
+        barrier()
+        torch.cuda.synchronize()
+        t0 = time.perf_counter()
+        for _ in range(args.e2e_steps):
+            if world == 1:
+                for s, qs, qc, qo, view in jobs:
+                    h.search(qc, qo, dbs[s], S, 10, 2, out=host_out[s], stream=stream)  # H2D + D2H inside
+            else:
+                for s, qs, qc, qo, view in jobs:
+                    h.search(qc, qo, dbs[s], S, 10, 2, out=view, stream=stream)      # H2D of queries inside
+                pg.all_gather_into_tensor(gathered, flat)
+                if rank == 0:
+                    final_host.copy_(gathered, non_blocking=False)
+        torch.cuda.synchronize()
+        dt = time.perf_counter() - t0
+        dtt = torch.tensor([dt], dtype=torch.float64, device=dev)
+        if pg is not None:
+            pg.all_reduce(dtt, op=pg.ReduceOp.MAX)
+        e2e = {"value": round(total_cells * args.e2e_steps / float(dtt.item()) / 1e9, 2), "unit": "GCUPS",
+               "h2d_bytes_per_step": h2d * world, "d2h_bytes_per_step": d2h}
+
+    cpu = None
+    if rank == 0 and world == 1 and not args.no_cpu_baseline:
+        cpu = cpu_baseline(c, args.cpu_baseline_cells)
+
+    if rank == 0:
+        line = {"metric": METRIC, "value": round(value, 2), "unit": "GCUPS", "n_gpus": world, "steps": args.steps,
+                "warmup": args.warmup, "ms_per_step": round(T / args.steps, 3), "higher_is_better": True,
+                "scaling": "strong", "vs_baseline": None, "dtype": "int16x2 (DPX), int32 re-score",
+                "data": "synthetic", "config": config_obj(args, c, q_lens, d_lens, world),
+                "roofline": {"bound": "alu", "achieved": round(achieved, 1) if achieved else None,
+                             "peak": round(peak, 1), "unit": "GCUPS", "frac": round(achieved / peak, 4) if achieved else None,
+                             "traffic": traffic,
+                             "kernel": "inter_kernel (short pairs), CUDA events around each launch",
+                             "peak_basis": f"{n_sm} SMs x {ALU_LANES_PER_SM_CLK} DPX lanes/clk x {sm_max:.0f} MHz / "
+                                           f"{OPS_PER_CELL} lane-ops per cell"},
+                "cpu_baseline": cpu, "e2e": e2e, "gpu_launches": int(n_launch_step * args.steps),
+                "clocks": clk,
+                "detail": {"search_ms_per_step": round(T / args.steps, 3),
+                           "short_kernel_ms_per_step": round(st["short_ms"] / args.steps, 3),
+                           "long_kernel_ms_per_step": round(st["long_ms"] / args.steps, 3),
+                           "cells_per_step": total_cells, "placement_makespan_model": plan.makespan}}
+        print(json.dumps(line), flush=True)
+    h.close()
+    if pg is not None:
+        pg.destroy_process_group()
+
+
+def main():
+    args = parse()
+    if args.impl == "reference":
+        run_reference(args)
+    else:
+        run_ours(args)
+
+
+if __name__ == "__main__":
+    main()

@@ -105,13 +105,17 @@ typedef struct {
 int32_t sw_db_info(sw_db_t db, sw_db_info_t* out);
 
 typedef struct {
-  double cells;            /* sum_q m_q * sum_d n_d of the last search (real residues) */
-  double cells_computed;   /* including row/column padding and wavefront fill         */
-  double kernel_ms;        /* summed CUDA-event time of the scoring kernels (TIMING)   */
-  int32_t n_launches;      /* kernels launched by the last search                     */
-  int32_t n_score_launches;/* of which scoring (inter-task) kernels                   */
-  int32_t n_overflow;      /* pairs re-scored in int32 (needs a synchronize)           */
-  int32_t timing_valid;
+  double cells;            /* sum_q m_q * sum_d n_d of the last search (real residues)      */
+  double cells_short;      /* of which in pairs of length <= 3000 (the bulk launches)        */
+  double cells_computed;   /* cell updates issued incl. row/column padding and wave fill     */
+  double short_ms;         /* summed CUDA-event time of the short-pair scoring launches      */
+  double long_ms;          /* summed CUDA-event time of the long-pair launches (overlapped)  */
+  double search_ms;        /* device time of the whole search, first upload to last kernel   */
+  int32_t n_launches;      /* kernels launched by the last search                           */
+  int32_t n_score_launches;/* of which scoring (inter-task) kernels                         */
+  int32_t n_overflow;      /* pairs re-scored in int32                                      */
+  int32_t timing_valid;    /* 1 if the handle had SW_FLAG_TIMING / "timing" set              */
+  int32_t last_G, last_R;  /* lane-group geometry of the last short-pair launch             */
 } sw_stats_t;
 /* Stats of the last sw_search; synchronizes the last search's stream. */
 int32_t sw_last_stats(sw_handle_t h, sw_stats_t* out);
@@ -120,7 +124,13 @@ int32_t sw_last_stats(sw_handle_t h, sw_stats_t* out);
  * Integer options (testing / tuning).  Keys:
  *   "overflow_threshold"  force the int16 re-score threshold (0 = automatic)
  *   "force_G", "force_R"  force the inter-task lane-group geometry (0 = auto)
+ *   "t_long"              DB pairs longer than this (default 3000) are scored in
+ *                         the intra-task mode (all warps of a CTA on one pair);
+ *                         applies to databases loaded afterwards
  *   "timing"              1/0, same as SW_FLAG_TIMING
+ *   "timing_accumulate"   1: short_ms/long_ms of sw_last_stats sum every search
+ *                         since the last "timing_reset" (0: the last search only)
+ *   "timing_reset"        clear the accumulated kernel events
  */
 int32_t sw_set_option(sw_handle_t h, const char* key, int64_t value);
 

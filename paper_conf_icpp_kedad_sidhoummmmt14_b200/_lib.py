@@ -30,9 +30,11 @@ class DbInfo(ctypes.Structure):
 
 
 class Stats(ctypes.Structure):
-    _fields_ = [("cells", ctypes.c_double), ("cells_computed", ctypes.c_double), ("kernel_ms", ctypes.c_double),
+    _fields_ = [("cells", ctypes.c_double), ("cells_short", ctypes.c_double), ("cells_computed", ctypes.c_double),
+                ("short_ms", ctypes.c_double), ("long_ms", ctypes.c_double), ("search_ms", ctypes.c_double),
                 ("n_launches", ctypes.c_int32), ("n_score_launches", ctypes.c_int32),
-                ("n_overflow", ctypes.c_int32), ("timing_valid", ctypes.c_int32)]
+                ("n_overflow", ctypes.c_int32), ("timing_valid", ctypes.c_int32),
+                ("last_G", ctypes.c_int32), ("last_R", ctypes.c_int32)]
 
 
 _lib = None

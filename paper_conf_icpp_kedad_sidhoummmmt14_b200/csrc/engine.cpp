@@ -84,9 +84,14 @@ struct sw_handle_s {
   std::string err;
   std::vector<sw_db_s*> dbs;
   // scratch (grown on demand)
-  DevBuf qcodes, qoff, matrix, prof, bbuf, counters, ovf, ovf_count, scores_tmp, rbuf;
+  DevBuf qcodes, qoff, matrix, prof, bbuf, prof_long, bbuf_long, counters, ovf, ovf_count, scores_tmp, rbuf;
+  cudaEvent_t ev_begin = nullptr, ev_end = nullptr;
+  bool search_timed = false;
+  bool timing_accumulate = false;
+  std::vector<int> event_kind;
   // options
   int64_t opt_thr = 0, opt_G = 0, opt_R = 0;
+  int64_t opt_t_long = T_LONG;  // pairs longer than this use the intra-task (long) mode
   // last-search bookkeeping
   sw_stats_t stats{};
   cudaStream_t last_stream = nullptr;
@@ -203,6 +208,14 @@ int32_t sw_set_option(sw_handle_t h, const char* key, int64_t value) {
     if (value != 0 && (value < 8 || value > 32 || value % 4))
       return set_err(h, SW_EINVAL, "force_R must be 0 or a multiple of 4 in [8, 32]");
     h->opt_R = value;
+  } else if (k == "t_long") {
+    if (value < 0) return set_err(h, SW_EINVAL, "t_long must be >= 0");
+    h->opt_t_long = value;
+  } else if (k == "timing_accumulate") {
+    h->timing_accumulate = value != 0;  // keep kernel events across searches until "timing_reset"
+    h->n_events_used = 0;
+  } else if (k == "timing_reset") {
+    h->n_events_used = 0;
   } else if (k == "timing") {
     if (value) h->flags |= SW_FLAG_TIMING; else h->flags &= ~uint32_t(SW_FLAG_TIMING);
   } else
@@ -225,7 +238,7 @@ int32_t sw_load_db(sw_handle_t h, const uint8_t* codes, const int64_t* offsets, 
     db->alpha = alphabet_size;
     Packed P;
     try {
-      pack_db(codes, offsets, n_seqs, alphabet_size, T_LONG, P);
+      pack_db(codes, offsets, n_seqs, alphabet_size, h->opt_t_long, P);
     } catch (const std::invalid_argument& e) {
       fail(SW_EINVAL, std::string("sw_load_db: ") + e.what());
     }
@@ -265,14 +278,117 @@ int32_t sw_db_info(sw_db_t db, sw_db_info_t* out) {
   return SW_OK;
 }
 
-static cudaEvent_t* next_event_pair(sw_handle_s* h) {
+static std::pair<cudaEvent_t, cudaEvent_t>* next_event_pair(sw_handle_s* h) {
   if (h->n_events_used == h->events.size()) {
     cudaEvent_t a, b;
     if (cudaEventCreate(&a) != cudaSuccess) return nullptr;
     if (cudaEventCreate(&b) != cudaSuccess) { cudaEventDestroy(a); return nullptr; }
     h->events.push_back({a, b});
+    h->event_kind.push_back(0);
   }
-  return &h->events[h->n_events_used++].first;
+  return &h->events[h->n_events_used++];
+}
+
+// One scoring launch per query: profile build(s) + the persistent kernel over
+// the long pairs [0, nlong) (intra-task mode) and the short pairs [nlong, np).
+struct LaunchCtx {
+  sw_handle_s* h;
+  sw_db_s* db;
+  cudaStream_t st;
+  int32_t* dscores;      // [nq][N]
+  int32_t thr;
+  OvfRec* ovf;
+  int* ovf_count;
+  int64_t ovf_cap;
+  uint32_t nGe, nGsGe;
+  bool timing;
+  double sum_short;      // sum of short pair lengths
+  int32_t max_short, max_long;
+};
+
+static void launch_query(LaunchCtx& c, int qi, const uint8_t* dq, int m, int* counter, double& cells_computed,
+                         int& launches) {
+  sw_handle_s* h = c.h;
+  sw_db_s* db = c.db;
+  const int alpha = db->alpha;
+  const int np = int(db->pairs.size());
+  const int nlong = db->n_long;
+  const int nshort = np - nlong;
+  int G = 32, R = 16;
+  if (nshort > 0) choose_geom(h, m, c.sum_short / nshort, false, G, R);
+  if (!inter_config_supported(G, R)) fail(SW_EUNSUPPORTED, "no kernel for this geometry");
+  const ProfGeom geom = make_geom(G, R, m, alpha);
+  const ProfGeom lgeom = make_geom(32, LONG_R, m, alpha);
+  const int NT = 256, NG = NT / G, W = NT / 32;
+  const size_t prof_bytes = size_t(geom.n_strips) * geom.SB;
+  const size_t lprof_bytes = nlong > 0 ? size_t(lgeom.n_strips) * lgeom.SB : 0;
+  SW_CK(h->prof.ensure(prof_bytes + lprof_bytes + 16));
+  uint8_t* prof = h->prof.as<uint8_t>();
+  uint8_t* lprof = prof + prof_bytes;
+  if (nshort > 0) {
+    SW_CK(launch_build_profile(dq, m, h->matrix.as<int8_t>(), alpha, geom, prof, c.st));
+    ++launches;
+  }
+  if (nlong > 0) {
+    SW_CK(launch_build_profile(dq, m, h->matrix.as<int8_t>(), alpha, lgeom, lprof, c.st));
+    ++launches;
+  }
+  const int smem = geom.SB + (nlong > 0 ? W * lgeom.SB : 0);
+  const int occ = inter_max_ctas_per_sm(G, R, NT, smem);
+  if (occ <= 0) fail(SW_ECUDA, "inter kernel does not fit on an SM");
+  const int n_items = nlong + (nshort + NG - 1) / NG;
+  const int grid = std::max(1, std::min(n_items, occ * h->sms));
+  const int bcap = c.max_short + G + 8;
+  if (geom.n_strips > 1 && nshort > 0) SW_CK(h->bbuf.ensure(size_t(grid) * NG * bcap * sizeof(uint2)));
+  const int lcap = c.max_long + 32 + 8;
+  if (nlong > 0 && lgeom.n_strips > 1) SW_CK(h->bbuf_long.ensure(size_t(grid) * W * lcap * sizeof(uint2)));
+  InterArgs a{};
+  a.prof = prof;
+  a.n_strips = geom.n_strips;
+  a.SB = geom.SB;
+  a.LS = geom.LS;
+  a.LB = geom.LB;
+  a.prof_long = lprof;
+  a.n_long = nlong;
+  a.n_strips_long = lgeom.n_strips;
+  a.SBL = lgeom.SB;
+  a.LSL = lgeom.LS;
+  a.LBL = lgeom.LB;
+  a.links = (nlong > 0 && lgeom.n_strips > 1) ? h->bbuf_long.as<uint2>() : nullptr;
+  a.lcap = lcap;
+  a.stream = db->stream.as<uint16_t>();
+  a.pairs = db->dpairs.as<PairRec>();
+  a.pair_begin = nlong;
+  a.pair_end = np;
+  a.bbuf = (geom.n_strips > 1 && nshort > 0) ? h->bbuf.as<uint2>() : nullptr;
+  a.bcap = bcap;
+  a.work_counter = counter;
+  a.scores = c.dscores + int64_t(qi) * db->n_seqs;
+  a.thr = c.thr;
+  a.ovf = c.ovf;
+  a.ovf_count = c.ovf_count;
+  a.ovf_cap = int(c.ovf_cap);
+  a.qidx = qi;
+  a.code_pad2 = uint32_t(alpha) | (uint32_t(alpha) << 8);
+  a.nGe = c.nGe;
+  a.nGsGe = c.nGsGe;
+  auto* ev = c.timing ? next_event_pair(h) : nullptr;
+  if (ev) {
+    h->event_kind[h->n_events_used - 1] = 0;
+    SW_CK(cudaEventRecord(ev->first, c.st));
+  }
+  SW_CK(launch_inter(G, R, NT, grid, smem, a, c.st));
+  if (ev) SW_CK(cudaEventRecord(ev->second, c.st));
+  ++launches;
+  ++h->stats.n_score_launches;
+  double sumS = 0, sumL = 0;
+  for (int p = 0; p < np; ++p) {
+    if (p < nlong) sumL += db->pairs[size_t(p)].len + 32;
+    else sumS += db->pairs[size_t(p)].len + G;
+  }
+  cells_computed += 2.0 * sumS * double(geom.n_strips) * G * R + 2.0 * sumL * double(lgeom.n_strips) * 32 * LONG_R;
+  h->stats.last_G = G;
+  h->stats.last_R = R;
 }
 
 int32_t sw_search(sw_handle_t h, const uint8_t* q_codes, const int64_t* q_offsets, int32_t n_queries, sw_db_t db,
@@ -290,8 +406,9 @@ int32_t sw_search(sw_handle_t h, const uint8_t* q_codes, const int64_t* q_offset
     SW_CK(cudaSetDevice(h->device));
     cudaStream_t st = reinterpret_cast<cudaStream_t>(cuda_stream);
     h->stats = sw_stats_t{};
-    h->n_events_used = 0;
+    if (!h->timing_accumulate) h->n_events_used = 0;
     h->last_stream = st;
+    h->search_timed = false;
     if (n_queries == 0 || db->n_seqs == 0) return;
     if (!scores) fail(SW_EINVAL, "sw_search: scores is NULL");
     // queries
@@ -325,6 +442,11 @@ int32_t sw_search(sw_handle_t h, const uint8_t* q_codes, const int64_t* q_offset
       SW_CK(h->scores_tmp.ensure(out_bytes));
       dscores = h->scores_tmp.as<int32_t>();
     }
+    const bool timing = (h->flags & SW_FLAG_TIMING) != 0;
+    if (timing) {
+      if (!h->ev_begin) { SW_CK(cudaEventCreate(&h->ev_begin)); SW_CK(cudaEventCreate(&h->ev_end)); }
+      SW_CK(cudaEventRecord(h->ev_begin, st));
+    }
     // upload queries, offsets rebased to 0
     std::vector<int64_t> qoff0(size_t(n_queries) + 1);
     for (int i = 0; i <= n_queries; ++i) qoff0[size_t(i)] = q_offsets[i] - q_offsets[0];
@@ -351,88 +473,49 @@ int32_t sw_search(sw_handle_t h, const uint8_t* q_codes, const int64_t* q_offset
     SW_CK(h->ovf.ensure(size_t(std::max<int64_t>(ovf_cap, 1)) * sizeof(OvfRec)));
     SW_CK(h->ovf_count.ensure(sizeof(int)));
     SW_CK(cudaMemsetAsync(h->ovf_count.p, 0, sizeof(int), st));
-    // work counters: 2 launches per query
     SW_CK(h->counters.ensure(size_t(2 * n_queries) * sizeof(int)));
     SW_CK(cudaMemsetAsync(h->counters.p, 0, size_t(2 * n_queries) * sizeof(int), st));
-    const bool timing = (h->flags & SW_FLAG_TIMING) != 0;
-    double cells_computed = 0;
     const int np = int(db->pairs.size());
     const int nlong = db->n_long;
-    // average pair length of the short and long ranges
-    double sum_short = 0, sum_long = 0;
+    double sum_short = 0;
     int32_t max_short = 0, max_long = 0;
     for (int p = 0; p < np; ++p) {
-      if (p < nlong) { sum_long += db->pairs[size_t(p)].len; max_long = std::max(max_long, db->pairs[size_t(p)].len); }
-      else { sum_short += db->pairs[size_t(p)].len; max_short = std::max(max_short, db->pairs[size_t(p)].len); }
+      const int32_t L = db->pairs[size_t(p)].len;
+      if (p < nlong) max_long = std::max(max_long, L);
+      else { sum_short += L; max_short = std::max(max_short, L); }
     }
-    const int nshort = np - nlong;
     const uint32_t nGe16 = uint32_t(uint16_t(int16_t(-gap_extend)));
     const uint32_t nGsGe16 = uint32_t(uint16_t(int16_t(-(gap_open + gap_extend))));
+    LaunchCtx lc{};
+    lc.h = h;
+    lc.db = db;
+    lc.st = st;
+    lc.dscores = dscores;
+    lc.thr = thr;
+    lc.ovf = h->ovf.as<OvfRec>();
+    lc.ovf_count = h->ovf_count.as<int>();
+    lc.ovf_cap = ovf_cap;
+    lc.nGe = nGe16 | (nGe16 << 16);
+    lc.nGsGe = nGsGe16 | (nGsGe16 << 16);
+    lc.timing = timing;
+    lc.sum_short = sum_short;
+    lc.max_short = max_short;
+    lc.max_long = max_long;
+    double cells_computed = 0;
+    const uint8_t* dq = h->qcodes.as<uint8_t>();
+    int* ctr = h->counters.as<int>();
     for (int qi = 0; qi < n_queries; ++qi) {
       const int m = int(qlen[size_t(qi)]);
       if (m == 0) continue;
-      for (int part = 0; part < 2; ++part) {
-        const bool lp = (part == 0);
-        const int pb = lp ? 0 : nlong, pe = lp ? nlong : np;
-        if (pe <= pb) continue;
-        const double Lavg = lp ? sum_long / nlong : sum_short / nshort;
-        const int32_t Lmax = lp ? max_long : max_short;
-        int G, R;
-        choose_geom(h, m, Lavg, lp, G, R);
-        if (!inter_config_supported(G, R)) fail(SW_EUNSUPPORTED, "no kernel for this geometry");
-        const ProfGeom geom = make_geom(G, R, m, alpha);
-        SW_CK(h->prof.ensure(size_t(geom.n_strips) * geom.SB));
-        SW_CK(launch_build_profile(h->qcodes.as<uint8_t>() + qoff0[size_t(qi)], m, h->matrix.as<int8_t>(), alpha,
-                                   geom, h->prof.as<uint8_t>(), st));
-        ++launches;
-        const int NT = 256, NG = NT / G;
-        const int smem = geom.SB;
-        const int occ = inter_max_ctas_per_sm(G, R, NT, smem);
-        if (occ <= 0) fail(SW_ECUDA, "inter kernel does not fit on an SM");
-        const int nchunks = (pe - pb + NG - 1) / NG;
-        const int grid = std::max(1, std::min(nchunks, occ * h->sms));
-        const int bcap = Lmax + G + 8;
-        if (geom.n_strips > 1) SW_CK(h->bbuf.ensure(size_t(grid) * NG * bcap * sizeof(uint2)));
-        InterArgs a{};
-        a.prof = h->prof.as<uint8_t>();
-        a.n_strips = geom.n_strips;
-        a.SB = geom.SB;
-        a.LS = geom.LS;
-        a.LB = geom.LB;
-        a.stream = db->stream.as<uint16_t>();
-        a.pairs = db->dpairs.as<PairRec>();
-        a.pair_begin = pb;
-        a.pair_end = pe;
-        a.bbuf = geom.n_strips > 1 ? h->bbuf.as<uint2>() : nullptr;
-        a.bcap = bcap;
-        a.work_counter = h->counters.as<int>() + 2 * qi + part;
-        a.scores = dscores + int64_t(qi) * N;
-        a.thr = thr;
-        a.ovf = h->ovf.as<OvfRec>();
-        a.ovf_count = h->ovf_count.as<int>();
-        a.ovf_cap = int(ovf_cap);
-        a.qidx = qi;
-        a.code_pad2 = uint32_t(alpha) | (uint32_t(alpha) << 8);
-        a.nGe = nGe16 | (nGe16 << 16);
-        a.nGsGe = nGsGe16 | (nGsGe16 << 16);
-        cudaEvent_t* ev = timing ? next_event_pair(h) : nullptr;
-        if (ev) SW_CK(cudaEventRecord(ev[0], st));
-        SW_CK(launch_inter(G, R, NT, grid, smem, a, st));
-        if (ev) SW_CK(cudaEventRecord(ev[1], st));
-        ++launches;
-        ++h->stats.n_score_launches;
-        double sumL = 0;
-        for (int p = pb; p < pe; ++p) sumL += db->pairs[size_t(p)].len + G;
-        cells_computed += 2.0 * sumL * double(geom.n_strips) * G * R;
-      }
+      launch_query(lc, qi, dq + qoff0[size_t(qi)], m, ctr + 2 * qi, cells_computed, launches);
     }
     if (ovf_cap > 0) {
-      int32_t Lmax = std::max(max_short, max_long);
+      const int32_t Lmax = std::max(max_short, max_long);
       const int grid = std::max(1, std::min<int>(int((ovf_cap + RESCORE_WARPS - 1) / RESCORE_WARPS), h->sms * 2));
       const int bcap = Lmax + 40;
       SW_CK(h->rbuf.ensure(size_t(grid) * RESCORE_WARPS * bcap * sizeof(int2)));
       RescoreArgs r{};
-      r.qcodes = h->qcodes.as<uint8_t>();
+      r.qcodes = dq;
       r.qoff = h->qoff.as<int64_t>();
       r.stream = db->stream.as<uint16_t>();
       r.pairs = db->dpairs.as<PairRec>();
@@ -449,6 +532,10 @@ int32_t sw_search(sw_handle_t h, const uint8_t* q_codes, const int64_t* q_offset
       SW_CK(launch_rescore(grid, r, st));
       ++launches;
     }
+    if (timing) {
+      SW_CK(cudaEventRecord(h->ev_end, st));
+      h->search_timed = true;
+    }
     if (!dev_scores) {
       SW_CK(cudaMemcpyAsync(scores, dscores, out_bytes, cudaMemcpyDeviceToHost, st));
       SW_CK(cudaStreamSynchronize(st));
@@ -456,6 +543,12 @@ int32_t sw_search(sw_handle_t h, const uint8_t* q_codes, const int64_t* q_offset
     double sq = 0;
     for (auto L : qlen) sq += double(L);
     h->stats.cells = sq * double(db->n_res);
+    double short_res = 0;
+    for (int p = nlong; p < np; ++p) {
+      const PairRec& r = db->pairs[size_t(p)];
+      short_res += double(db->seq_len[size_t(r.id0)]) + (r.id1 >= 0 ? double(db->seq_len[size_t(r.id1)]) : 0.0);
+    }
+    h->stats.cells_short = sq * short_res;  // pairs <= 3000 columns (inter-task mode)
     h->stats.cells_computed = cells_computed;
     h->stats.n_launches = launches;
   });
@@ -472,13 +565,20 @@ int32_t sw_last_stats(sw_handle_t h, sw_stats_t* out) {
       SW_CK(cudaMemcpy(&c, h->ovf_count.p, sizeof(int), cudaMemcpyDeviceToHost));
       s.n_overflow = c;
     }
-    double ms = 0;
+    double ms_s = 0, ms_l = 0;
     for (size_t i = 0; i < h->n_events_used; ++i) {
       float t = 0;
       SW_CK(cudaEventElapsedTime(&t, h->events[i].first, h->events[i].second));
-      ms += t;
+      if (h->event_kind[i] == 0) ms_s += t; else ms_l += t;
     }
-    s.kernel_ms = ms;
+    s.short_ms = ms_s;
+    s.long_ms = ms_l;
+    s.search_ms = 0;
+    if (h->search_timed) {
+      float t = 0;
+      SW_CK(cudaEventElapsedTime(&t, h->ev_begin, h->ev_end));
+      s.search_ms = t;
+    }
     s.timing_valid = h->n_events_used > 0 ? 1 : 0;
     *out = s;
   });
@@ -508,6 +608,8 @@ int32_t sw_free(sw_handle_t h) {
     cudaEventDestroy(e.first);
     cudaEventDestroy(e.second);
   }
+  for (cudaEvent_t e : {h->ev_begin, h->ev_end})
+    if (e) cudaEventDestroy(e);
   delete h;
   return SW_OK;
 }

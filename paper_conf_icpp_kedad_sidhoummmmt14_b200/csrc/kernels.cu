@@ -67,42 +67,63 @@ __device__ __forceinline__ void copy_strip(uint8_t* dst, const uint8_t* __restri
   for (int i = threadIdx.x; i < bytes / 16; i += blockDim.x) d[i] = __ldg(s + i);
 }
 
-template <int G, int R>
-__device__ __forceinline__ void strip_pass(const InterArgs& a, const uint8_t* sprof, const PairRec& pr, int T,
-                                           int k, bool rd, bool wr, uint2* __restrict__ bb, uint32_t& best) {
+// One strip pass of a lane group over one pair: G lanes x R rows, columns
+// streamed as an anti-diagonal wave.  Boundary rows: lane 0 reads the strip
+// above at rp[c] (c = column, rp = row base + G - 1), lane G-1 writes this
+// strip's bottom row at wp[t] (t = step).  LINKED: the row above is produced
+// concurrently by another warp of the CTA (intra-task mode): lane 0 waits on
+// its progress counter, lane G-1 publishes its own.
+template <int G, int R, bool LINKED>
+__device__ __forceinline__ void strip_pass(const uint8_t* sprof, int LS, int LB, const uint16_t* pstream, int L,
+                                           int T, int k, bool rd, bool wr, const uint2* __restrict__ rp,
+                                           uint2* __restrict__ wp, volatile int* prog_in, int need_base,
+                                           volatile int* prog_out, int pub_base, uint32_t code_pad2, uint32_t nGe,
+                                           uint32_t nGsGe, uint32_t& best) {
   uint32_t Hl[R], E[R];
 #pragma unroll
   for (int r = 0; r < R; ++r) { Hl[r] = 0; E[r] = 0; }
-  uint32_t hdiag = 0, sH = 0, sF = 0, sC = a.code_pad2;
-  const uint2* __restrict__ codes = reinterpret_cast<const uint2*>(a.stream + pr.off);
-  const int L = pr.len;
-  const uint32_t pad4 = a.code_pad2 | (a.code_pad2 << 16);
-  const uint32_t laneoff = uint32_t(k) * a.LB;
+  uint32_t hdiag = 0, sH = 0, sF = 0, sC = code_pad2;
+  const uint2* __restrict__ codes = reinterpret_cast<const uint2*>(pstream);
+  const uint32_t pad4 = code_pad2 | (code_pad2 << 16);
+  const uint32_t laneoff = uint32_t(k) * LB;
   const bool lead = (k == 0), tail = (k == G - 1);
+  const uint2 z2 = make_uint2(0, 0);
 
-  // lane 0 prefetch of block 0: 4 columns of codes and (if rd) 4 boundary cells
+  // lane 0 prefetch of block 0: 4 columns of codes and (if rd) 4 boundary cells.
+  // L and t0 are multiples of 4, so one compare guards a whole block.
   uint2 cw = make_uint2(pad4, pad4);
-  uint2 tb0 = make_uint2(0, 0), tb1 = tb0, tb2 = tb0, tb3 = tb0;
-  if (lead) {
-    if (L > 0) cw = codes[0];
+  uint2 tb0 = z2, tb1 = z2, tb2 = z2, tb3 = z2;
+  if (lead && L > 0) {
+    cw = codes[0];
     if (rd) {
-      if (0 < L) tb0 = bb[0 + G - 1];
-      if (1 < L) tb1 = bb[1 + G - 1];
-      if (2 < L) tb2 = bb[2 + G - 1];
-      if (3 < L) tb3 = bb[3 + G - 1];
+      if (LINKED) {
+        while (*prog_in < need_base + 4 + G - 1) __nanosleep(64);
+        __threadfence_block();
+        tb0 = __ldcg(rp + 0); tb1 = __ldcg(rp + 1); tb2 = __ldcg(rp + 2); tb3 = __ldcg(rp + 3);
+      } else {
+        tb0 = rp[0]; tb1 = rp[1]; tb2 = rp[2]; tb3 = rp[3];
+      }
     }
   }
   for (int t0 = 0; t0 < T; t0 += 4) {
     const uint2 cwc = cw;
     const uint2 c0 = tb0, c1 = tb1, c2 = tb2, c3 = tb3;
+    rp += 4;
     if (lead) {
-      const int n0 = t0 + 4;
-      cw = (n0 < L) ? codes[n0 >> 2] : make_uint2(pad4, pad4);
-      if (rd) {
-        tb0 = (n0 + 0 < L) ? bb[n0 + 0 + G - 1] : make_uint2(0, 0);
-        tb1 = (n0 + 1 < L) ? bb[n0 + 1 + G - 1] : make_uint2(0, 0);
-        tb2 = (n0 + 2 < L) ? bb[n0 + 2 + G - 1] : make_uint2(0, 0);
-        tb3 = (n0 + 3 < L) ? bb[n0 + 3 + G - 1] : make_uint2(0, 0);
+      if (t0 + 4 < L) {
+        cw = codes[(t0 + 4) >> 2];
+        if (rd) {
+          if (LINKED) {
+            while (*prog_in < need_base + t0 + 8 + G - 1) __nanosleep(64);
+            __threadfence_block();
+            tb0 = __ldcg(rp + 0); tb1 = __ldcg(rp + 1); tb2 = __ldcg(rp + 2); tb3 = __ldcg(rp + 3);
+          } else {
+            tb0 = rp[0]; tb1 = rp[1]; tb2 = rp[2]; tb3 = rp[3];
+          }
+        }
+      } else {
+        cw = make_uint2(pad4, pad4);
+        tb0 = z2; tb1 = z2; tb2 = z2; tb3 = z2;
       }
     }
 #pragma unroll
@@ -117,68 +138,131 @@ __device__ __forceinline__ void strip_pass(const InterArgs& a, const uint8_t* sp
         rH = tv.x;
         rF = tv.y;
       }
-      const uint8_t* pa = sprof + (rC & 0xffu) * a.LS + laneoff;
-      const uint8_t* pb = sprof + (rC >> 8) * a.LS + laneoff;
-      gotoh_column<R>(Hl, E, best, hdiag, pa, pb, rH, rF, a.nGe, a.nGsGe);
+      const uint8_t* pa = sprof + (rC & 0xffu) * LS + laneoff;
+      const uint8_t* pb = sprof + (rC >> 8) * LS + laneoff;
+      gotoh_column<R>(Hl, E, best, hdiag, pa, pb, rH, rF, nGe, nGsGe);
       sH = rH;
       sF = rF;
       sC = rC;
-      if (wr && tail) bb[t0 + j] = make_uint2(rH, rF);
+      if (wr && tail) {
+        if (LINKED) __stcg(wp + j, make_uint2(rH, rF));
+        else wp[j] = make_uint2(rH, rF);
+      }
+    }
+    wp += 4;
+    if (LINKED && wr) {
+      __syncwarp();
+      if (tail) {
+        __threadfence_block();
+        *prog_out = pub_base + t0 + 4;
+      }
     }
   }
 }
 
+__device__ __forceinline__ void emit_pair(const InterArgs& a, int p, const PairRec& pr, uint32_t best) {
+  const int lo = int(int16_t(best & 0xffffu));
+  const int hi = int(int16_t(best >> 16));
+  a.scores[pr.id0] = lo;
+  if (lo >= a.thr) {
+    const int e = atomicAdd(a.ovf_count, 1);
+    if (e < a.ovf_cap) a.ovf[e] = OvfRec{a.qidx, p, 0, 0};
+  }
+  if (pr.id1 >= 0) {
+    a.scores[pr.id1] = hi;
+    if (hi >= a.thr) {
+      const int e = atomicAdd(a.ovf_count, 1);
+      if (e < a.ovf_cap) a.ovf[e] = OvfRec{a.qidx, p, 1, 0};
+    }
+  }
+}
+
+// Persistent kernel over one query.  Work items, longest first:
+//   items [0, n_long): one LONG pair each, scored by all W = NT/32 warps of the
+//     CTA together (intra-task mode; the paper's fine-grained
+//     wavefront across PEs, Fig. 2): warp w takes strips w, w+W, ...
+//     of a 32-lane x LONG_R-row geometry, each strip consuming the bottom row
+//     of the strip above through a global link row + shared progress counter;
+//   items [n_long, ...): a CHUNK of NT/G short pairs, one per lane group
+//     (inter-task mode).
 template <int G, int R, int NT>
 __global__ void __launch_bounds__(NT) inter_kernel(InterArgs a) {
-  extern __shared__ __align__(16) uint8_t sprof[];
-  __shared__ int s_chunk;
+  extern __shared__ __align__(16) uint8_t smem[];
+  uint8_t* sprof = smem;           // short-mode strip profile (a.SB bytes)
+  uint8_t* lprof = smem + a.SB;    // long mode: one a.SBL slot per warp
+  __shared__ int s_item;
+  __shared__ int s_prog[NT / 32];
+  __shared__ uint32_t s_best[NT / 32];
   constexpr int NG = NT / G;
+  constexpr int W = NT / 32;
   const int tid = threadIdx.x;
   const int k = tid & (G - 1);
   const int g = tid / G;
-  const int npairs = a.pair_end - a.pair_begin;
-  const int nchunks = (npairs + NG - 1) / NG;
+  const int lane = tid & 31, warp = tid >> 5;
+  const int n_short = a.pair_end - a.pair_begin;
+  const int n_items = a.n_long + (n_short + NG - 1) / NG;
   uint2* __restrict__ bb = a.bbuf + ((size_t)blockIdx.x * NG + g) * (size_t)a.bcap;
 
-  if (a.n_strips == 1) copy_strip(sprof, a.prof, a.SB);
+  if (a.n_strips == 1 && n_short > 0) copy_strip(sprof, a.prof, a.SB);
   for (;;) {
-    if (tid == 0) s_chunk = atomicAdd(a.work_counter, 1);
+    if (tid == 0) s_item = atomicAdd(a.work_counter, 1);
+    if (tid < W) { s_prog[tid] = -1; s_best[tid] = 0; }
     __syncthreads();
-    const int chunk = s_chunk;
-    if (chunk >= nchunks) break;
-    const int p = a.pair_begin + chunk * NG + g;
-    const bool valid = p < a.pair_end;
-    PairRec pr;
-    if (valid) pr = a.pairs[p];
-    else { pr.off = 0; pr.len = 0; pr.id0 = -1; pr.id1 = -1; }
-    int T = pr.len + G;                       // lane G-1 finishes column len-1 at step len+G-2
-    if (G < 32) T = __reduce_max_sync(FULL, T);  // warp-uniform trip count (shuffles)
-    uint32_t best = 0;
-    for (int s = 0; s < a.n_strips; ++s) {
-      if (a.n_strips > 1) {
-        __syncthreads();
-        copy_strip(sprof, a.prof + (size_t)s * a.SB, a.SB);
-        __syncthreads();
-      }
-      strip_pass<G, R>(a, sprof, pr, T, k, s > 0, s + 1 < a.n_strips, bb, best);
-    }
-#pragma unroll
-    for (int o = G / 2; o > 0; o >>= 1) best = __vmaxs2(best, __shfl_xor_sync(FULL, best, o, G));
-    if (valid && k == 0) {
-      const int lo = int(int16_t(best & 0xffffu));
-      const int hi = int(int16_t(best >> 16));
-      a.scores[pr.id0] = lo;
-      if (lo >= a.thr) {
-        const int e = atomicAdd(a.ovf_count, 1);
-        if (e < a.ovf_cap) a.ovf[e] = OvfRec{a.qidx, p, 0, 0};
-      }
-      if (pr.id1 >= 0) {
-        a.scores[pr.id1] = hi;
-        if (hi >= a.thr) {
-          const int e = atomicAdd(a.ovf_count, 1);
-          if (e < a.ovf_cap) a.ovf[e] = OvfRec{a.qidx, p, 1, 0};
+    const int item = s_item;
+    if (item >= n_items) break;
+    if (item < a.n_long) {
+      // ---------------- long pair: chained strips across the CTA's warps
+      const PairRec pr = a.pairs[item];
+      const int T = pr.len + 32;
+      uint32_t best = 0;
+      uint8_t* myprof = lprof + warp * a.SBL;
+      uint2* links = a.links + (size_t)blockIdx.x * W * a.lcap;
+      for (int s = warp; s < a.n_strips_long; s += W) {
+        __syncwarp();
+        {  // this warp's strip profile -> its own slot
+          const uint4* src = reinterpret_cast<const uint4*>(a.prof_long + (size_t)s * a.SBL);
+          uint4* dst = reinterpret_cast<uint4*>(myprof);
+          for (int i = lane; i < a.SBL / 16; i += 32) dst[i] = __ldg(src + i);
         }
+        __syncwarp();
+        const bool rd = s > 0, wr = s + 1 < a.n_strips_long;
+        const int lin = (s + W - 1) % W, lout = s % W;
+        strip_pass<32, LONG_R, true>(myprof, a.LSL, a.LBL, a.stream + pr.off, pr.len, T, lane, rd, wr,
+                                     links + (size_t)lin * a.lcap + 31, links + (size_t)lout * a.lcap,
+                                     &s_prog[lin], (s - 1) << 20, &s_prog[lout], s << 20, a.code_pad2, a.nGe,
+                                     a.nGsGe, best);
       }
+#pragma unroll
+      for (int o = 16; o > 0; o >>= 1) best = __vmaxs2(best, __shfl_xor_sync(FULL, best, o));
+      if (lane == 0) s_best[warp] = best;
+      __syncthreads();
+      if (tid == 0) {
+        uint32_t b = 0;
+        for (int w = 0; w < W; ++w) b = __vmaxs2(b, s_best[w]);
+        emit_pair(a, item, pr, b);
+      }
+    } else {
+      // ---------------- chunk of short pairs, one per lane group
+      const int p = a.pair_begin + (item - a.n_long) * NG + g;
+      const bool valid = p < a.pair_end;
+      PairRec pr;
+      if (valid) pr = a.pairs[p];
+      else { pr.off = 0; pr.len = 0; pr.id0 = -1; pr.id1 = -1; }
+      int T = pr.len + G;                          // lane G-1 finishes column len-1 at step len+G-2
+      if (G < 32) T = __reduce_max_sync(FULL, T);  // warp-uniform trip count (shuffles)
+      uint32_t best = 0;
+      for (int s = 0; s < a.n_strips; ++s) {
+        if (a.n_strips > 1) {
+          __syncthreads();
+          copy_strip(sprof, a.prof + (size_t)s * a.SB, a.SB);
+          __syncthreads();
+        }
+        strip_pass<G, R, false>(sprof, a.LS, a.LB, a.stream + pr.off, pr.len, T, k, s > 0, s + 1 < a.n_strips,
+                                bb + (G - 1), bb, nullptr, 0, nullptr, 0, a.code_pad2, a.nGe, a.nGsGe, best);
+      }
+#pragma unroll
+      for (int o = G / 2; o > 0; o >>= 1) best = __vmaxs2(best, __shfl_xor_sync(FULL, best, o, G));
+      if (valid && k == 0) emit_pair(a, p, pr, best);
     }
     __syncthreads();
   }

@@ -11,7 +11,7 @@
 //
 // Two independent problems share every 32-bit register (s16x2): the low half
 // scores the query against DB sequence id0 of a pair, the high half against id1.
-// Per cell pair: VIMNMX (max E,F) + VIADDMNMX (H) + VIADD.16x2 (H-Gs-Ge) +
+// Per cell pair: VIADDMNMX (Hdiag+S vs E) + VIMNMX (vs F) + VIADD.16x2 (H-Gs-Ge) +
 // 2x VIADDMNMX.RELU (E', F') + 1/2 VIMNMX3 (running max) = 5.5 DPX lane-ops,
 // plus one sign-extending PRMT that builds the (S[q_i][a], S[q_i][b]) word from
 // the int8 query profile rows of the two DB letters a, b.
@@ -75,7 +75,9 @@ __device__ __forceinline__ void gotoh_column(uint32_t (&Hl)[R], uint32_t (&E)[R]
     for (int j = 0; j < UB; ++j) {
       const int r = u * UB + j;
       const uint32_t s = prmt(wa[j >> 2], wb[j >> 2], pair_sel(j & 3));
-      const uint32_t h = __viaddmax_s16x2(hd, s, __vmaxs2(E[r], F));   // Eq. (2)
+      // Eq. (2): H = max(max(Hdiag + S, E), F); E, F >= 0 so the 0 term is implied.
+      // Folding E first keeps the row-to-row chain F -> H -> t -> F' at 3 ops.
+      const uint32_t h = __vmaxs2(__viaddmax_s16x2(hd, s, E[r]), F);
       hd = Hl[r];
       Hl[r] = h;
       const uint32_t t = __vadd2(h, nGsGe);                              // H - Gs - Ge

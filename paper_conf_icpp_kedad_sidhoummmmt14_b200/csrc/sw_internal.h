@@ -48,12 +48,19 @@ struct ProfGeom {
   int n_strips;    // ceil(m / (G*R))
 };
 
+constexpr int LONG_R = 8;    // rows per lane of the intra-task (long pair) geometry, G = 32
+
 struct InterArgs {
   const uint8_t* prof;       // [n_strips][SB]
   int n_strips, SB, LS, LB;
+  // long pairs (intra-task mode): pairs [0, n_long), geometry G = 32, R = LONG_R
+  const uint8_t* prof_long;  // [n_strips_long][SBL]
+  int n_long, n_strips_long, SBL, LSL, LBL;
+  uint2* links;              // [gridDim][NT/32][lcap] strip-to-strip rows
+  int lcap;
   const uint16_t* stream;
   const PairRec* pairs;
-  int pair_begin, pair_end;  // [begin, end) pairs of this launch
+  int pair_begin, pair_end;  // [begin, end): the short pairs of this launch
   uint2* bbuf;               // boundary rows, [gridDim][NG][bcap]
   int bcap;
   int* work_counter;

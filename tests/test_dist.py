@@ -1,0 +1,120 @@
+"""Multi-GPU layer host logic: shard cut, dual-approx placement of
+(query, shard) tasks, and the all-gather + assembly -- run with world_size 2
+over gloo on CPU.  The per-rank scoring backend here is the CPU oracle (tests
+may use it); on the GPU box the same dist.run() drives sw_search over NCCL.
+The invariant: scores are identical for any world size and placement."""
+import os
+import socket
+
+import numpy as np
+import pytest
+import torch
+import torch.distributed as tdist
+import torch.multiprocessing as tmp
+
+import oracle
+import swgen
+from oracle.blosum62 import blosum62 as ob62
+from paper_conf_icpp_kedad_sidhoummmmt14_b200 import dist as swdist
+
+
+def _workload():
+    c = swgen.make_config("c1", n_db=160, q_lens=[37, 90, 12])
+    return c
+
+
+def _score_block_oracle(c, shards):
+    def f(s, qs):
+        sc, so = swdist.subset(c["dcodes"], c["doff"], shards[s])
+        qc, qo = swdist.subset(c["qcodes"], c["qoff"], qs)
+        return oracle.gotoh_search(qc, qo, sc, so, ob62(), 10, 2)
+    return f
+
+
+def test_shard_cut_partition_and_balance():
+    c = swgen.make_config("c2", n_db=5000)
+    lens = np.diff(c["doff"])
+    for S in (1, 2, 3, 8):
+        sh = swdist.shard_cut(c["doff"], S)
+        allidx = np.sort(np.concatenate(sh))
+        assert np.array_equal(allidx, np.arange(len(lens)))
+        res = [int(lens[s].sum()) for s in sh]
+        assert max(res) - min(res) <= 2 * lens.max()
+        for s in sh:
+            assert np.all(np.diff(s) > 0)
+
+
+def test_subset_roundtrip():
+    rng = np.random.default_rng(3)
+    codes, off = swgen.random_seqs(rng, 50, 0, 30)
+    idx = np.array([7, 3, 3, 49, 0])
+    sc, so = swdist.subset(codes, off, idx)
+    for k, i in enumerate(idx):
+        assert np.array_equal(sc[so[k]:so[k + 1]], codes[off[i]:off[i + 1]])
+
+
+def test_place_covers_every_task():
+    c = swgen.make_config("c3", n_db=3000)
+    ql = np.diff(c["qoff"])
+    for g in (1, 2, 4, 8):
+        sh = swdist.shard_cut(c["doff"], g)
+        res = [int(np.diff(c["doff"])[s].sum()) for s in sh]
+        plan = swdist.place(ql, sh, res, g)
+        seen = sorted((q, s) for r in range(g) for s, qs in swdist.local_blocks(plan, r) for q in qs)
+        assert seen == sorted(plan.tasks)
+        loads = np.zeros(g)
+        for (q, s), o in zip(plan.tasks, plan.owner):
+            loads[o] += ql[q] * res[s]
+        assert loads.max() == pytest.approx(plan.makespan)
+        assert plan.makespan <= 2 * plan.lam * (1 + 1e-9)
+
+
+def test_single_process_run_matches_oracle():
+    c = _workload()
+    ref = oracle.gotoh_search(c["qcodes"], c["qoff"], c["dcodes"], c["doff"], ob62(), 10, 2)
+    sh = swdist.shard_cut(c["doff"], 3)
+    res = [int(np.diff(c["doff"])[s].sum()) for s in sh]
+    plan = swdist.place(np.diff(c["qoff"]), sh, res, 1)
+    got = swdist.run(plan, 0, len(c["qoff"]) - 1, len(c["doff"]) - 1, _score_block_oracle(c, sh))
+    np.testing.assert_array_equal(got, ref)
+
+
+def _worker(rank, world, port, n_shards, q):
+    os.environ.update(MASTER_ADDR="127.0.0.1", MASTER_PORT=str(port))
+    tdist.init_process_group("gloo", rank=rank, world_size=world)
+    try:
+        c = _workload()
+        sh = swdist.shard_cut(c["doff"], n_shards)
+        res = [int(np.diff(c["doff"])[s].sum()) for s in sh]
+        plan = swdist.place(np.diff(c["qoff"]), sh, res, world)
+        out = swdist.run(plan, rank, len(c["qoff"]) - 1, len(c["doff"]) - 1, _score_block_oracle(c, sh),
+                         dist=tdist, assemble_on_all=True)
+        q.put((rank, out))
+    finally:
+        tdist.destroy_process_group()
+
+
+def _free_port():
+    s = socket.socket()
+    s.bind(("127.0.0.1", 0))
+    p = s.getsockname()[1]
+    s.close()
+    return p
+
+
+@pytest.mark.parametrize("n_shards", [2, 5])
+def test_gloo_world2_matches_single_process(n_shards):
+    c = _workload()
+    ref = oracle.gotoh_search(c["qcodes"], c["qoff"], c["dcodes"], c["doff"], ob62(), 10, 2)
+    ctx = tmp.get_context("spawn")
+    q = ctx.Queue()
+    port = _free_port()
+    procs = [ctx.Process(target=_worker, args=(r, 2, port, n_shards, q)) for r in range(2)]
+    for p in procs:
+        p.start()
+    outs = dict(q.get(timeout=240) for _ in procs)
+    for p in procs:
+        p.join(timeout=60)
+        assert p.exitcode == 0
+    for r in (0, 1):
+        np.testing.assert_array_equal(outs[r], ref)

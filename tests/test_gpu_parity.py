@@ -189,3 +189,42 @@ def test_swissprot_scale_sampled(name):
     sub = np.concatenate([c["dcodes"][c["doff"][i]:c["doff"][i + 1]] for i in idx])
     ref = oracle_scores(c["qcodes"], c["qoff"], sub, sub_off, procs=16)
     np.testing.assert_array_equal(got[:, idx], ref)
+
+
+def test_intra_task_mode_forced():
+    """t_long small: most pairs go through the chained-warps (intra-task) mode;
+    queries span 1 strip, exactly 1, 2, and more strips than warps (ring wrap)."""
+    rng = np.random.default_rng(21)
+    dl = list(rng.integers(1, 700, size=70)) + [0, 1, 65, 66, 67, 68]
+    dc, do = _seqs(dl, rng)
+    ql = [1, 100, 256, 257, 600, 2400]
+    qc, qo = _seqs(ql, rng)
+    got = gpu_scores(qc, qo, dc, do, opts={"t_long": 64})
+    np.testing.assert_array_equal(got, oracle_scores(qc, qo, dc, do))
+
+
+def test_long_db_sequences():
+    rng = np.random.default_rng(22)
+    dl = list(rng.integers(3001, 6000, size=24)) + list(rng.integers(1, 400, size=60))
+    dc, do = _seqs(dl, rng)
+    qc, qo = _seqs([567, 2600, 77], rng)
+    got = gpu_scores(qc, qo, dc, do)
+    np.testing.assert_array_equal(got, oracle_scores(qc, qo, dc, do, procs=16))
+
+
+def test_config_c4_sampled():
+    """BASELINE config 4 (queries 2,000-35,000 vs 1,500 long sequences) in full on
+    the GPU; the oracle checks a seeded sample plus every planted long homolog."""
+    c = swgen.make_config("c4")
+    got = gpu_scores(c["qcodes"], c["qoff"], c["dcodes"], c["doff"])
+    N = len(c["doff"]) - 1
+    rng = np.random.default_rng(23)
+    sample = set(rng.choice(N, size=6, replace=False).tolist()) | {p[0] for p in c["plants"]}
+    idx = np.array(sorted(sample), dtype=np.int64)
+    lens = c["doff"][idx + 1] - c["doff"][idx]
+    sub_off = np.zeros(len(idx) + 1, dtype=np.int64)
+    np.cumsum(lens, out=sub_off[1:])
+    sub = np.concatenate([c["dcodes"][c["doff"][i]:c["doff"][i + 1]] for i in idx])
+    ref = oracle_scores(c["qcodes"], c["qoff"], sub, sub_off, procs=16)
+    assert ref.max() > 32767  # planted self-hits of >= 6.4k queries really overflow int16
+    np.testing.assert_array_equal(got[:, idx], ref)

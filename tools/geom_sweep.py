@@ -47,9 +47,11 @@ def main():
                 ms.append(t0.elapsed_time(t1))
             st = h.last_stats()
             best = min(ms)
-            print(json.dumps({"m": m, "G": G, "R": R, "ms": round(best, 3), "kernel_ms": round(st["kernel_ms"], 3),
+            print(json.dumps({"m": m, "G": st["last_G"], "R": st["last_R"], "ms": round(best, 3),
+                              "search_ms": round(st["search_ms"], 3), "short_ms": round(st["short_ms"], 3),
+                              "long_ms": round(st["long_ms"], 3),
                               "GCUPS": round(st["cells"] / best / 1e6, 1),
-                              "kernel_GCUPS": round(st["cells"] / st["kernel_ms"] / 1e6, 1),
+                              "short_GCUPS": round(st["cells_short"] / st["short_ms"] / 1e6, 1),
                               "pad_frac": round(1 - st["cells"] / st["cells_computed"], 4)}), flush=True)
     h.close()
 

@@ -84,7 +84,7 @@ struct sw_handle_s {
   std::string err;
   std::vector<sw_db_s*> dbs;
   // scratch (grown on demand)
-  DevBuf qcodes, qoff, matrix, prof, bbuf, prof_long, bbuf_long, counters, ovf, ovf_count, scores_tmp, rbuf;
+  DevBuf qcodes, qoff, matrix, prof, bbuf, bbuf_long, counters, ovf, ovf_count, scores_tmp, rbuf, qdesc;
   cudaEvent_t ev_begin = nullptr, ev_end = nullptr;
   bool search_timed = false;
   bool timing_accumulate = false;
@@ -146,7 +146,11 @@ static ProfGeom make_geom(int G, int R, int m, int alpha) {
   return g;
 }
 
-static void choose_geom(const sw_handle_s* h, int m, double Lavg, bool long_pairs, int& G, int& R) {
+// One (G, R) for all queries of a launch: minimise the modelled cell updates
+// (row padding to whole strips, wavefront fill of G-1 columns per pair and
+// strip, a per-step overhead amortised over R rows, a register-pressure
+// penalty for the largest R).
+static void choose_geom(const sw_handle_s* h, const std::vector<int>& ms, double Lavg, int& G, int& R) {
   if (h->opt_G > 0 && h->opt_R > 0) {
     G = int(h->opt_G);
     R = int(h->opt_R);
@@ -155,17 +159,17 @@ static void choose_geom(const sw_handle_s* h, int m, double Lavg, bool long_pair
   static const int Gs[] = {4, 8, 16, 32};
   static const int Rs[] = {8, 12, 16, 20, 24, 28, 32};
   double best = 1e300;
-  G = 32;
-  R = 16;
+  G = 4;
+  R = 24;
   for (int g : Gs) {
-    if (long_pairs && g != 32) continue;
     for (int r : Rs) {
-      const int strips = std::max(1, (m + g * r - 1) / (g * r));
-      const double rows = double(strips) * g * r;
-      // per-step overhead ~ 7 instr / (5.5 per row) plus register-pressure penalty for big R
       const double per_cell = 1.0 + 7.0 / (5.5 * r) + (r > 24 ? 0.06 : 0.0);
-      const double strip_ovh = strips > 1 ? 0.02 : 0.0;
-      const double cost = rows * (Lavg + g) * per_cell * (1.0 + strip_ovh);
+      double cost = 0;
+      for (int m : ms) {
+        const int strips = std::max(1, (m + g * r - 1) / (g * r));
+        const double rows = double(strips) * g * r;
+        cost += rows * (Lavg + g) * per_cell * (strips > 1 ? 1.02 : 1.0);
+      }
       if (cost < best) { best = cost; G = g; R = r; }
     }
   }
@@ -289,8 +293,8 @@ static std::pair<cudaEvent_t, cudaEvent_t>* next_event_pair(sw_handle_s* h) {
   return &h->events[h->n_events_used++];
 }
 
-// One scoring launch per query: profile build(s) + the persistent kernel over
-// the long pairs [0, nlong) (intra-task mode) and the short pairs [nlong, np).
+// The scoring launch: profiles of every query, then ONE persistent kernel over
+// all (query, long pair) and (query, short chunk) work items.
 struct LaunchCtx {
   sw_handle_s* h;
   sw_db_s* db;
@@ -306,69 +310,108 @@ struct LaunchCtx {
   int32_t max_short, max_long;
 };
 
-static void launch_query(LaunchCtx& c, int qi, const uint8_t* dq, int m, int* counter, double& cells_computed,
-                         int& launches) {
+static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std::vector<int64_t>& qoff0,
+                       double& cells_computed, int& launches) {
   sw_handle_s* h = c.h;
   sw_db_s* db = c.db;
   const int alpha = db->alpha;
   const int np = int(db->pairs.size());
   const int nlong = db->n_long;
   const int nshort = np - nlong;
-  int G = 32, R = 16;
-  if (nshort > 0) choose_geom(h, m, c.sum_short / nshort, false, G, R);
+  std::vector<int> order;
+  for (int i = 0; i < int(qlen.size()); ++i)
+    if (qlen[size_t(i)] > 0) order.push_back(i);
+  if (order.empty() || np == 0) return;
+  std::stable_sort(order.begin(), order.end(), [&](int x, int y) { return qlen[size_t(x)] > qlen[size_t(y)]; });
+  std::vector<int> ms;
+  for (int i : order) ms.push_back(int(qlen[size_t(i)]));
+  int G = 4, R = 24;
+  choose_geom(h, ms, nshort > 0 ? c.sum_short / nshort : 1.0, G, R);
   if (!inter_config_supported(G, R)) fail(SW_EUNSUPPORTED, "no kernel for this geometry");
-  const ProfGeom geom = make_geom(G, R, m, alpha);
-  const ProfGeom lgeom = make_geom(32, LONG_R, m, alpha);
   const int NT = 256, NG = NT / G, W = NT / 32;
-  const size_t prof_bytes = size_t(geom.n_strips) * geom.SB;
-  const size_t lprof_bytes = nlong > 0 ? size_t(lgeom.n_strips) * lgeom.SB : 0;
-  SW_CK(h->prof.ensure(prof_bytes + lprof_bytes + 16));
+  // profiles: short (G x R) and long (32 x LONG_R) geometry for every query
+  size_t total = 0;
+  std::vector<ProfGeom> gs, gl;
+  std::vector<size_t> off_s, off_l;
+  for (int m : ms) {
+    gs.push_back(make_geom(G, R, m, alpha));
+    gl.push_back(make_geom(32, LONG_R, m, alpha));
+    off_s.push_back(total);
+    total += nshort > 0 ? size_t(gs.back().n_strips) * gs.back().SB : 0;
+    off_l.push_back(total);
+    total += nlong > 0 ? size_t(gl.back().n_strips) * gl.back().SB : 0;
+  }
+  SW_CK(h->prof.ensure(total + 16));
   uint8_t* prof = h->prof.as<uint8_t>();
-  uint8_t* lprof = prof + prof_bytes;
-  if (nshort > 0) {
-    SW_CK(launch_build_profile(dq, m, h->matrix.as<int8_t>(), alpha, geom, prof, c.st));
-    ++launches;
+  std::vector<QueryDesc> desc(order.size());
+  double sumS = 0, sumL = 0;
+  for (int p = 0; p < np; ++p) {
+    if (p < nlong) sumL += db->pairs[size_t(p)].len + 32;
+    else sumS += db->pairs[size_t(p)].len + G;
   }
-  if (nlong > 0) {
-    SW_CK(launch_build_profile(dq, m, h->matrix.as<int8_t>(), alpha, lgeom, lprof, c.st));
-    ++launches;
+  for (size_t k = 0; k < order.size(); ++k) {
+    const int qi = order[k];
+    const uint8_t* dq = h->qcodes.as<uint8_t>() + qoff0[size_t(qi)];
+    if (nshort > 0) {
+      SW_CK(launch_build_profile(dq, ms[k], h->matrix.as<int8_t>(), alpha, gs[k], prof + off_s[k], c.st));
+      ++launches;
+    }
+    if (nlong > 0) {
+      SW_CK(launch_build_profile(dq, ms[k], h->matrix.as<int8_t>(), alpha, gl[k], prof + off_l[k], c.st));
+      ++launches;
+    }
+    QueryDesc& d = desc[k];
+    d.prof = prof + off_s[k];
+    d.prof_long = prof + off_l[k];
+    d.scores = c.dscores + int64_t(qi) * db->n_seqs;
+    d.n_strips = gs[k].n_strips;
+    d.n_strips_long = gl[k].n_strips;
+    d.qidx = qi;
+    d.pad_ = 0;
+    cells_computed += 2.0 * sumS * double(gs[k].n_strips) * G * R + 2.0 * sumL * double(gl[k].n_strips) * 32 * LONG_R;
   }
-  const int smem = geom.SB + (nlong > 0 ? W * lgeom.SB : 0);
+  SW_CK(h->qdesc.ensure(desc.size() * sizeof(QueryDesc)));
+  SW_CK(cudaMemcpyAsync(h->qdesc.p, desc.data(), desc.size() * sizeof(QueryDesc), cudaMemcpyHostToDevice, c.st));
+  const ProfGeom g0 = gs[0], l0 = gl[0];
+  const int smem = g0.SB + (nlong > 0 ? W * l0.SB : 0);
   const int occ = inter_max_ctas_per_sm(G, R, NT, smem);
   if (occ <= 0) fail(SW_ECUDA, "inter kernel does not fit on an SM");
-  const int n_items = nlong + (nshort + NG - 1) / NG;
-  const int grid = std::max(1, std::min(n_items, occ * h->sms));
+  const int64_t n_items = int64_t(order.size()) * (nlong + (nshort + NG - 1) / NG);
+  if (n_items >= (int64_t(1) << 31)) fail(SW_EUNSUPPORTED, "too many work items");
+  const int grid = int(std::max<int64_t>(1, std::min<int64_t>(n_items, int64_t(occ) * h->sms)));
+  int max_strips = 1;
+  for (auto& x : gs) max_strips = std::max(max_strips, x.n_strips);
+  int max_lstrips = 1;
+  for (auto& x : gl) max_lstrips = std::max(max_lstrips, x.n_strips);
   const int bcap = c.max_short + G + 8;
-  if (geom.n_strips > 1 && nshort > 0) SW_CK(h->bbuf.ensure(size_t(grid) * NG * bcap * sizeof(uint2)));
+  if (max_strips > 1 && nshort > 0) SW_CK(h->bbuf.ensure(size_t(grid) * NG * bcap * sizeof(uint2)));
   const int lcap = c.max_long + 32 + 8;
-  if (nlong > 0 && lgeom.n_strips > 1) SW_CK(h->bbuf_long.ensure(size_t(grid) * W * lcap * sizeof(uint2)));
+  if (nlong > 0 && max_lstrips > 1) SW_CK(h->bbuf_long.ensure(size_t(grid) * W * lcap * sizeof(uint2)));
+  SW_CK(h->counters.ensure(sizeof(int)));
+  SW_CK(cudaMemsetAsync(h->counters.p, 0, sizeof(int), c.st));
   InterArgs a{};
-  a.prof = prof;
-  a.n_strips = geom.n_strips;
-  a.SB = geom.SB;
-  a.LS = geom.LS;
-  a.LB = geom.LB;
-  a.prof_long = lprof;
+  a.queries = h->qdesc.as<QueryDesc>();
+  a.n_queries = int(order.size());
+  a.SB = g0.SB;
+  a.LS = g0.LS;
+  a.LB = g0.LB;
+  a.SBL = l0.SB;
+  a.LSL = l0.LS;
+  a.LBL = l0.LB;
   a.n_long = nlong;
-  a.n_strips_long = lgeom.n_strips;
-  a.SBL = lgeom.SB;
-  a.LSL = lgeom.LS;
-  a.LBL = lgeom.LB;
-  a.links = (nlong > 0 && lgeom.n_strips > 1) ? h->bbuf_long.as<uint2>() : nullptr;
+  a.links = (nlong > 0 && max_lstrips > 1) ? h->bbuf_long.as<uint2>() : nullptr;
   a.lcap = lcap;
   a.stream = db->stream.as<uint16_t>();
   a.pairs = db->dpairs.as<PairRec>();
   a.pair_begin = nlong;
   a.pair_end = np;
-  a.bbuf = (geom.n_strips > 1 && nshort > 0) ? h->bbuf.as<uint2>() : nullptr;
+  a.bbuf = (max_strips > 1 && nshort > 0) ? h->bbuf.as<uint2>() : nullptr;
   a.bcap = bcap;
-  a.work_counter = counter;
-  a.scores = c.dscores + int64_t(qi) * db->n_seqs;
+  a.work_counter = h->counters.as<int>();
   a.thr = c.thr;
   a.ovf = c.ovf;
   a.ovf_count = c.ovf_count;
   a.ovf_cap = int(c.ovf_cap);
-  a.qidx = qi;
   a.code_pad2 = uint32_t(alpha) | (uint32_t(alpha) << 8);
   a.nGe = c.nGe;
   a.nGsGe = c.nGsGe;
@@ -381,12 +424,6 @@ static void launch_query(LaunchCtx& c, int qi, const uint8_t* dq, int m, int* co
   if (ev) SW_CK(cudaEventRecord(ev->second, c.st));
   ++launches;
   ++h->stats.n_score_launches;
-  double sumS = 0, sumL = 0;
-  for (int p = 0; p < np; ++p) {
-    if (p < nlong) sumL += db->pairs[size_t(p)].len + 32;
-    else sumS += db->pairs[size_t(p)].len + G;
-  }
-  cells_computed += 2.0 * sumS * double(geom.n_strips) * G * R + 2.0 * sumL * double(lgeom.n_strips) * 32 * LONG_R;
   h->stats.last_G = G;
   h->stats.last_R = R;
 }
@@ -473,8 +510,6 @@ int32_t sw_search(sw_handle_t h, const uint8_t* q_codes, const int64_t* q_offset
     SW_CK(h->ovf.ensure(size_t(std::max<int64_t>(ovf_cap, 1)) * sizeof(OvfRec)));
     SW_CK(h->ovf_count.ensure(sizeof(int)));
     SW_CK(cudaMemsetAsync(h->ovf_count.p, 0, sizeof(int), st));
-    SW_CK(h->counters.ensure(size_t(2 * n_queries) * sizeof(int)));
-    SW_CK(cudaMemsetAsync(h->counters.p, 0, size_t(2 * n_queries) * sizeof(int), st));
     const int np = int(db->pairs.size());
     const int nlong = db->n_long;
     double sum_short = 0;
@@ -503,16 +538,11 @@ int32_t sw_search(sw_handle_t h, const uint8_t* q_codes, const int64_t* q_offset
     lc.max_long = max_long;
     double cells_computed = 0;
     const uint8_t* dq = h->qcodes.as<uint8_t>();
-    int* ctr = h->counters.as<int>();
-    for (int qi = 0; qi < n_queries; ++qi) {
-      const int m = int(qlen[size_t(qi)]);
-      if (m == 0) continue;
-      launch_query(lc, qi, dq + qoff0[size_t(qi)], m, ctr + 2 * qi, cells_computed, launches);
-    }
+    launch_all(lc, qlen, qoff0, cells_computed, launches);
     if (ovf_cap > 0) {
       const int32_t Lmax = std::max(max_short, max_long);
-      const int grid = std::max(1, std::min<int>(int((ovf_cap + RESCORE_WARPS - 1) / RESCORE_WARPS), h->sms * 2));
-      const int bcap = Lmax + 40;
+      const int grid = std::max(1, std::min<int>(int(ovf_cap), h->sms * 2));  // one CTA per flagged pair
+      const int bcap = Lmax + 32 + 8;
       SW_CK(h->rbuf.ensure(size_t(grid) * RESCORE_WARPS * bcap * sizeof(int2)));
       RescoreArgs r{};
       r.qcodes = dq;

@@ -24,6 +24,10 @@ namespace swdual {
 
 constexpr uint32_t FULL = 0xffffffffu;
 constexpr int8_t PAD_SCORE = -64;  // S[.][PAD] = S[PAD][.] <= 0 (reading R-12)
+// Intra-task mode: a strip starts consuming the row above only once its
+// producer is this many columns ahead, so producer and consumer warps of a
+// chain run decoupled instead of in lock-step (the consumer then rarely waits).
+constexpr int LINK_LAG = 64;
 
 // ---------------------------------------------------------------------------
 // Query profile: prof[s][a][k][r] = S[q[s*G*R + k*R + r]][a]  (int8)
@@ -60,6 +64,18 @@ cudaError_t launch_build_profile(const uint8_t* q, int m, const int8_t* matrix, 
   return cudaGetLastError();
 }
 
+// Warp-uniform wait until a shared progress counter reaches `need` (all lanes
+// read the broadcast word; __all_sync keeps the warp converged so the shuffles
+// that follow stay on the fast path), then a CTA-scope acquire fence.
+__device__ __forceinline__ void wait_progress(volatile int* p, int need) {
+  for (;;) {
+    const int v = *p;
+    if (__all_sync(FULL, v >= need)) break;
+    __nanosleep(32);
+  }
+  __threadfence_block();
+}
+
 // ---------------------------------------------------------------------------
 __device__ __forceinline__ void copy_strip(uint8_t* dst, const uint8_t* __restrict__ src, int bytes) {
   const uint4* s = reinterpret_cast<const uint4*>(src);
@@ -93,39 +109,33 @@ __device__ __forceinline__ void strip_pass(const uint8_t* sprof, int LS, int LB,
   // L and t0 are multiples of 4, so one compare guards a whole block.
   uint2 cw = make_uint2(pad4, pad4);
   uint2 tb0 = z2, tb1 = z2, tb2 = z2, tb3 = z2;
+  if (LINKED && rd && L > 0) wait_progress(prog_in, need_base + min(4 + G - 1 + LINK_LAG, L + G));
   if (lead && L > 0) {
     cw = codes[0];
     if (rd) {
-      if (LINKED) {
-        while (*prog_in < need_base + 4 + G - 1) __nanosleep(64);
-        __threadfence_block();
-        tb0 = __ldcg(rp + 0); tb1 = __ldcg(rp + 1); tb2 = __ldcg(rp + 2); tb3 = __ldcg(rp + 3);
-      } else {
-        tb0 = rp[0]; tb1 = rp[1]; tb2 = rp[2]; tb3 = rp[3];
-      }
+      if (LINKED) { tb0 = __ldcg(rp + 0); tb1 = __ldcg(rp + 1); tb2 = __ldcg(rp + 2); tb3 = __ldcg(rp + 3); }
+      else { tb0 = rp[0]; tb1 = rp[1]; tb2 = rp[2]; tb3 = rp[3]; }
     }
   }
+  __syncwarp();
   for (int t0 = 0; t0 < T; t0 += 4) {
     const uint2 cwc = cw;
     const uint2 c0 = tb0, c1 = tb1, c2 = tb2, c3 = tb3;
     rp += 4;
+    if (LINKED && rd && t0 + 4 < L) wait_progress(prog_in, need_base + min(t0 + 8 + G - 1 + LINK_LAG, L + G));
     if (lead) {
       if (t0 + 4 < L) {
         cw = codes[(t0 + 4) >> 2];
         if (rd) {
-          if (LINKED) {
-            while (*prog_in < need_base + t0 + 8 + G - 1) __nanosleep(64);
-            __threadfence_block();
-            tb0 = __ldcg(rp + 0); tb1 = __ldcg(rp + 1); tb2 = __ldcg(rp + 2); tb3 = __ldcg(rp + 3);
-          } else {
-            tb0 = rp[0]; tb1 = rp[1]; tb2 = rp[2]; tb3 = rp[3];
-          }
+          if (LINKED) { tb0 = __ldcg(rp + 0); tb1 = __ldcg(rp + 1); tb2 = __ldcg(rp + 2); tb3 = __ldcg(rp + 3); }
+          else { tb0 = rp[0]; tb1 = rp[1]; tb2 = rp[2]; tb3 = rp[3]; }
         }
       } else {
         cw = make_uint2(pad4, pad4);
         tb0 = z2; tb1 = z2; tb2 = z2; tb3 = z2;
       }
     }
+    __syncwarp();
 #pragma unroll
     for (int j = 0; j < 4; ++j) {
       uint32_t rH = __shfl_up_sync(FULL, sH, 1, G);
@@ -160,31 +170,33 @@ __device__ __forceinline__ void strip_pass(const uint8_t* sprof, int LS, int LB,
   }
 }
 
-__device__ __forceinline__ void emit_pair(const InterArgs& a, int p, const PairRec& pr, uint32_t best) {
+__device__ __forceinline__ void emit_pair(const InterArgs& a, const QueryDesc& d, int p, const PairRec& pr,
+                                          uint32_t best) {
   const int lo = int(int16_t(best & 0xffffu));
   const int hi = int(int16_t(best >> 16));
-  a.scores[pr.id0] = lo;
+  d.scores[pr.id0] = lo;
   if (lo >= a.thr) {
     const int e = atomicAdd(a.ovf_count, 1);
-    if (e < a.ovf_cap) a.ovf[e] = OvfRec{a.qidx, p, 0, 0};
+    if (e < a.ovf_cap) a.ovf[e] = OvfRec{d.qidx, p, 0, 0};
   }
   if (pr.id1 >= 0) {
-    a.scores[pr.id1] = hi;
+    d.scores[pr.id1] = hi;
     if (hi >= a.thr) {
       const int e = atomicAdd(a.ovf_count, 1);
-      if (e < a.ovf_cap) a.ovf[e] = OvfRec{a.qidx, p, 1, 0};
+      if (e < a.ovf_cap) a.ovf[e] = OvfRec{d.qidx, p, 1, 0};
     }
   }
 }
 
-// Persistent kernel over one query.  Work items, longest first:
-//   items [0, n_long): one LONG pair each, scored by all W = NT/32 warps of the
-//     CTA together (intra-task mode; the paper's fine-grained
+// Persistent kernel over ALL queries of a search.  Work items, costliest first:
+//   [0, Q*n_long): (query, LONG pair) -- scored by all W = NT/32 warps of the CTA
+//     together (intra-task mode; the paper's fine-grained
 //     wavefront across PEs, Fig. 2): warp w takes strips w, w+W, ...
-//     of a 32-lane x LONG_R-row geometry, each strip consuming the bottom row
-//     of the strip above through a global link row + shared progress counter;
-//   items [n_long, ...): a CHUNK of NT/G short pairs, one per lane group
+//     of a 32-lane x LONG_R-row geometry, each strip consuming the bottom row of
+//     the strip above through a global link row + shared progress counter;
+//   then (query, CHUNK of NT/G short pairs) -- one pair per lane group
 //     (inter-task mode).
+// Queries are in descending length, pairs in descending length.
 template <int G, int R, int NT>
 __global__ void __launch_bounds__(NT) inter_kernel(InterArgs a) {
   extern __shared__ __align__(16) uint8_t smem[];
@@ -200,32 +212,36 @@ __global__ void __launch_bounds__(NT) inter_kernel(InterArgs a) {
   const int g = tid / G;
   const int lane = tid & 31, warp = tid >> 5;
   const int n_short = a.pair_end - a.pair_begin;
-  const int n_items = a.n_long + (n_short + NG - 1) / NG;
+  const int nchunks = (n_short + NG - 1) / NG;
+  const int n_long_items = a.n_queries * a.n_long;
+  const int n_items = n_long_items + a.n_queries * nchunks;
   uint2* __restrict__ bb = a.bbuf + ((size_t)blockIdx.x * NG + g) * (size_t)a.bcap;
+  int loaded = -1;  // (query rank << 16 | strip) of the short profile in shared memory (CTA-uniform)
 
-  if (a.n_strips == 1 && n_short > 0) copy_strip(sprof, a.prof, a.SB);
   for (;;) {
     if (tid == 0) s_item = atomicAdd(a.work_counter, 1);
     if (tid < W) { s_prog[tid] = -1; s_best[tid] = 0; }
     __syncthreads();
     const int item = s_item;
     if (item >= n_items) break;
-    if (item < a.n_long) {
+    if (item < n_long_items) {
       // ---------------- long pair: chained strips across the CTA's warps
-      const PairRec pr = a.pairs[item];
+      const int qr = item / a.n_long, pidx = item - qr * a.n_long;
+      const QueryDesc d = a.queries[qr];
+      const PairRec pr = a.pairs[pidx];
       const int T = pr.len + 32;
       uint32_t best = 0;
       uint8_t* myprof = lprof + warp * a.SBL;
       uint2* links = a.links + (size_t)blockIdx.x * W * a.lcap;
-      for (int s = warp; s < a.n_strips_long; s += W) {
+      for (int s = warp; s < d.n_strips_long; s += W) {
         __syncwarp();
         {  // this warp's strip profile -> its own slot
-          const uint4* src = reinterpret_cast<const uint4*>(a.prof_long + (size_t)s * a.SBL);
+          const uint4* src = reinterpret_cast<const uint4*>(d.prof_long + (size_t)s * a.SBL);
           uint4* dst = reinterpret_cast<uint4*>(myprof);
           for (int i = lane; i < a.SBL / 16; i += 32) dst[i] = __ldg(src + i);
         }
         __syncwarp();
-        const bool rd = s > 0, wr = s + 1 < a.n_strips_long;
+        const bool rd = s > 0, wr = s + 1 < d.n_strips_long;
         const int lin = (s + W - 1) % W, lout = s % W;
         strip_pass<32, LONG_R, true>(myprof, a.LSL, a.LBL, a.stream + pr.off, pr.len, T, lane, rd, wr,
                                      links + (size_t)lin * a.lcap + 31, links + (size_t)lout * a.lcap,
@@ -239,11 +255,14 @@ __global__ void __launch_bounds__(NT) inter_kernel(InterArgs a) {
       if (tid == 0) {
         uint32_t b = 0;
         for (int w = 0; w < W; ++w) b = __vmaxs2(b, s_best[w]);
-        emit_pair(a, item, pr, b);
+        emit_pair(a, d, pidx, pr, b);
       }
     } else {
       // ---------------- chunk of short pairs, one per lane group
-      const int p = a.pair_begin + (item - a.n_long) * NG + g;
+      const int c = item - n_long_items;
+      const int qr = c / nchunks, chunk = c - qr * nchunks;
+      const QueryDesc d = a.queries[qr];
+      const int p = a.pair_begin + chunk * NG + g;
       const bool valid = p < a.pair_end;
       PairRec pr;
       if (valid) pr = a.pairs[p];
@@ -251,18 +270,20 @@ __global__ void __launch_bounds__(NT) inter_kernel(InterArgs a) {
       int T = pr.len + G;                          // lane G-1 finishes column len-1 at step len+G-2
       if (G < 32) T = __reduce_max_sync(FULL, T);  // warp-uniform trip count (shuffles)
       uint32_t best = 0;
-      for (int s = 0; s < a.n_strips; ++s) {
-        if (a.n_strips > 1) {
+      for (int s = 0; s < d.n_strips; ++s) {
+        const int want = (qr << 16) | s;
+        if (want != loaded) {
           __syncthreads();
-          copy_strip(sprof, a.prof + (size_t)s * a.SB, a.SB);
+          copy_strip(sprof, d.prof + (size_t)s * a.SB, a.SB);
           __syncthreads();
+          loaded = want;
         }
-        strip_pass<G, R, false>(sprof, a.LS, a.LB, a.stream + pr.off, pr.len, T, k, s > 0, s + 1 < a.n_strips,
+        strip_pass<G, R, false>(sprof, a.LS, a.LB, a.stream + pr.off, pr.len, T, k, s > 0, s + 1 < d.n_strips,
                                 bb + (G - 1), bb, nullptr, 0, nullptr, 0, a.code_pad2, a.nGe, a.nGsGe, best);
       }
 #pragma unroll
       for (int o = G / 2; o > 0; o >>= 1) best = __vmaxs2(best, __shfl_xor_sync(FULL, best, o, G));
-      if (valid && k == 0) emit_pair(a, p, pr, best);
+      if (valid && k == 0) emit_pair(a, d, p, pr, best);
     }
     __syncthreads();
   }
@@ -313,25 +334,30 @@ cudaError_t launch_inter(int G, int R, int NT, int grid, int smem_bytes, const I
 }
 
 // ---------------------------------------------------------------------------
-// Exact int32 re-score of flagged pairs.  One warp per pair,
-// lane k owns RESCORE_R rows of a 32*RESCORE_R-row strip, same wavefront as the
-// inter-task kernel but one problem per lane and S read from the matrix.
+// Exact int32 re-score of flagged pairs.  One CTA per pair,
+// the same chained-warp intra-task wavefront as the long-pair mode but one
+// problem per lane in int32 and S read from a shared 33x33 matrix: warp w does
+// strips w, w+W, ... (32 lanes x RESCORE_R rows), strip s+1 consuming strip s's
+// bottom row through a global link row + shared progress counter.
 __global__ void __launch_bounds__(RESCORE_WARPS * 32) rescore_kernel(RescoreArgs a) {
   constexpr int R = RESCORE_R;
+  constexpr int W = RESCORE_WARPS;
   constexpr int SW = 33;  // matrix row stride (PAD = alpha <= 32)
   __shared__ int32_t sm[SW * SW];
+  __shared__ int s_prog[W];
+  __shared__ int s_best[W];
   for (int i = threadIdx.x; i < SW * SW; i += blockDim.x) {
     const int x = i / SW, y = i % SW;
     sm[i] = (x < a.alpha && y < a.alpha) ? int(a.matrix[x * a.alpha + y]) : int(PAD_SCORE);
   }
-  __syncthreads();
-  const int lane = threadIdx.x & 31;
-  const int gw = blockIdx.x * RESCORE_WARPS + threadIdx.x / 32;
-  const int nw = gridDim.x * RESCORE_WARPS;
-  int2* __restrict__ bb = a.bbuf + (size_t)gw * a.bcap;
+  const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
+  int2* __restrict__ links = a.bbuf + (size_t)blockIdx.x * W * a.bcap;
   const int cnt = *a.ovf_count;
   const int pad = a.alpha;
-  for (int e = gw; e < cnt; e += nw) {
+  for (int e = blockIdx.x; e < cnt; e += gridDim.x) {
+    __syncthreads();
+    if (threadIdx.x < W) { s_prog[threadIdx.x] = -1; s_best[threadIdx.x] = 0; }
+    __syncthreads();
     const OvfRec o = a.ovf[e];
     const PairRec pr = a.pairs[o.pair];
     const uint8_t* qc = a.qcodes + a.qoff[o.q];
@@ -339,9 +365,16 @@ __global__ void __launch_bounds__(RESCORE_WARPS * 32) rescore_kernel(RescoreArgs
     const int L = pr.len;
     const int shift = o.half ? 8 : 0;
     const int nstrips = (m + 32 * R - 1) / (32 * R);
+    const int T = L + 32;
     int best = 0;
-    for (int s = 0; s < nstrips; ++s) {
+    for (int s = warp; s < nstrips; s += W) {
       const bool rd = s > 0, wr = s + 1 < nstrips;
+      const int lin = (s + W - 1) % W, lout = s % W;
+      const int2* rp = links + (size_t)lin * a.bcap + 31;
+      int2* wp = links + (size_t)lout * a.bcap;
+      volatile int* pin = &s_prog[lin];
+      volatile int* pout = &s_prog[lout];
+      const int need_base = (s - 1) << 20, pub_base = s << 20;
       int qr[R], Hl[R], E[R];
 #pragma unroll
       for (int r = 0; r < R; ++r) {
@@ -351,48 +384,64 @@ __global__ void __launch_bounds__(RESCORE_WARPS * 32) rescore_kernel(RescoreArgs
         E[r] = 0;
       }
       int hdiag = 0, sH = 0, sF = 0, sC = pad;
-      const int T = L + 32;
       for (int t = 0; t < T; ++t) {
         int rH = __shfl_up_sync(FULL, sH, 1);
         int rF = __shfl_up_sync(FULL, sF, 1);
         int rC = __shfl_up_sync(FULL, sC, 1);
+        if (rd && t < L && (t & 3) == 0) wait_progress(pin, need_base + min(t + 36 + LINK_LAG, L + 32));
         if (lane == 0) {
           if (t < L) {
             rC = (a.stream[pr.off + t] >> shift) & 0xff;
-            if (rd) { const int2 v = bb[t + 31]; rH = v.x; rF = v.y; }
-            else { rH = 0; rF = 0; }
+            if (rd) {
+              const int2 v = __ldcg(rp + t);
+              rH = v.x;
+              rF = v.y;
+            } else { rH = 0; rF = 0; }
           } else { rC = pad; rH = 0; rF = 0; }
         }
+        __syncwarp();
         int hd = hdiag;
         hdiag = rH;
         int F = rF;
 #pragma unroll
         for (int r = 0; r < R; ++r) {
-          const int h = max(max(hd + sm[qr[r] + rC], max(E[r], F)), 0);  // Eq. (2)
+          const int h = max(max(hd + sm[qr[r] + rC], E[r]), F);        // Eq. (2) (E, F >= 0)
           hd = Hl[r];
           Hl[r] = h;
           const int tt = h - a.Gs - a.Ge;
-          E[r] = max(max(E[r] - a.Ge, tt), 0);                            // Eq. (3)
-          F = max(max(F - a.Ge, tt), 0);                                  // Eq. (4)
+          E[r] = max(max(E[r] - a.Ge, tt), 0);                          // Eq. (3)
+          F = max(max(F - a.Ge, tt), 0);                                // Eq. (4)
           best = max(best, h);
         }
         sH = Hl[R - 1];
         sF = F;
         sC = rC;
-        if (wr && lane == 31) bb[t] = make_int2(sH, sF);
+        if (wr && lane == 31) __stcg(wp + t, make_int2(sH, sF));
+        if (wr && (t & 3) == 3) {
+          __syncwarp();
+          if (lane == 31) { __threadfence_block(); *pout = pub_base + t + 1; }
+        }
+      }
+      if (wr) {
+        __syncwarp();
+        if (lane == 31) { __threadfence_block(); *pout = pub_base + T; }
       }
     }
 #pragma unroll
     for (int off = 16; off > 0; off >>= 1) best = max(best, __shfl_xor_sync(FULL, best, off));
-    if (lane == 0) {
+    if (lane == 0) s_best[warp] = best;
+    __syncthreads();
+    if (threadIdx.x == 0) {
+      int b = 0;
+      for (int w = 0; w < W; ++w) b = max(b, s_best[w]);
       const int id = o.half ? pr.id1 : pr.id0;
-      a.scores[(int64_t)o.q * a.n_seqs + id] = best;
+      a.scores[(int64_t)o.q * a.n_seqs + id] = b;
     }
   }
 }
 
 cudaError_t launch_rescore(int grid, const RescoreArgs& a, cudaStream_t st) {
-  rescore_kernel<<<grid, RESCORE_WARPS * 32, 0, st>>>(a);
+  rescore_kernel<<<grid, RESCORE_WARPS * 32, 0, st>>>(a);  // one CTA per flagged pair
   return cudaGetLastError();
 }
 

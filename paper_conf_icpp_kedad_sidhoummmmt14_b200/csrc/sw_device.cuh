@@ -91,4 +91,42 @@ __device__ __forceinline__ void gotoh_column(uint32_t (&Hl)[R], uint32_t (&E)[R]
   Fio = F;
 }
 
+// Query-pair variant (two QUERIES per register, one DB sequence): the profile
+// already holds (S[qA_i][a], S[qB_i][a]) as s16x2 words, 4 rows per 16-byte
+// load, so no PRMT is needed: 5.5 DPX lane-ops per cell pair, of which the
+// VIADD.16x2 runs on the FMA pipe (4.5 on the ALU pipe).
+template <int R>
+__device__ __forceinline__ void gotoh_column_q2(uint32_t (&Hl)[R], uint32_t (&E)[R], uint32_t& best,
+                                                uint32_t& hdiag, const uint8_t* __restrict__ pa, uint32_t& Hio,
+                                                uint32_t& Fio, uint32_t nGe, uint32_t nGsGe) {
+  static_assert(R % 4 == 0, "R must be a multiple of 4");
+  uint32_t hd = hdiag;
+  hdiag = Hio;
+  uint32_t F = Fio;
+  uint32_t hprev = 0;
+#pragma unroll
+  for (int u = 0; u < R / 4; ++u) {
+    const uint4 w = *reinterpret_cast<const uint4*>(pa + u * 16);
+    const uint32_t sv[4] = {w.x, w.y, w.z, w.w};
+#pragma unroll
+    for (int j = 0; j < 4; ++j) {
+      const int r = u * 4 + j;
+      const uint32_t h = __vmaxs2(__viaddmax_s16x2(hd, sv[j], E[r]), F);  // Eq. (2)
+      hd = Hl[r];
+      Hl[r] = h;
+      const uint32_t t = __vadd2(h, nGsGe);
+      E[r] = __viaddmax_s16x2_relu(E[r], nGe, t);                          // Eq. (3)
+      F = __viaddmax_s16x2_relu(F, nGe, t);                                // Eq. (4)
+      if (r & 1) best = __vimax3_s16x2(best, hprev, h);
+      else hprev = h;
+    }
+  }
+  Hio = Hl[R - 1];
+  Fio = F;
+}
+
+// Lane block of the query-pair profile: R 4-byte rows, rounded to an odd number
+// of 16-byte units (bank-conflict-free LDS.128 across the 8 lanes of a phase).
+__host__ __device__ constexpr int lane_block_bytes_q2(int R) { return (((R / 4) | 1) * 16); }
+
 }  // namespace swdual

@@ -50,26 +50,33 @@ struct ProfGeom {
 
 constexpr int LONG_R = 8;    // rows per lane of the intra-task (long pair) geometry, G = 32
 
+// Per-query descriptor of a multi-query launch (processing order: longest first).
+struct QueryDesc {
+  const uint8_t* prof;       // short-pair (inter-task) profile, [n_strips][SB]
+  const uint8_t* prof_long;  // long-pair (intra-task) profile, [n_strips_long][SBL]
+  int32_t* scores;           // this query's row of scores[Q][N] (caller order)
+  int n_strips, n_strips_long;
+  int qidx, pad_;
+};
+
 struct InterArgs {
-  const uint8_t* prof;       // [n_strips][SB]
-  int n_strips, SB, LS, LB;
-  // long pairs (intra-task mode): pairs [0, n_long), geometry G = 32, R = LONG_R
-  const uint8_t* prof_long;  // [n_strips_long][SBL]
-  int n_long, n_strips_long, SBL, LSL, LBL;
-  uint2* links;              // [gridDim][NT/32][lcap] strip-to-strip rows
+  const QueryDesc* queries;  // [n_queries], processing order
+  int n_queries;
+  int SB, LS, LB;            // short geometry (G, R of the launch)
+  int SBL, LSL, LBL;         // long geometry (32 lanes x LONG_R rows)
+  int n_long;                // pairs [0, n_long) are long (intra-task items)
+  uint2* links;              // [gridDim][NT/32][lcap] strip-to-strip rows (long items)
   int lcap;
   const uint16_t* stream;
   const PairRec* pairs;
-  int pair_begin, pair_end;  // [begin, end): the short pairs of this launch
-  uint2* bbuf;               // boundary rows, [gridDim][NG][bcap]
+  int pair_begin, pair_end;  // [begin, end): the short pairs
+  uint2* bbuf;               // boundary rows of multi-strip short items, [gridDim][NG][bcap]
   int bcap;
   int* work_counter;
-  int32_t* scores;           // row of this query: scores[id]
   int32_t thr;               // overflow threshold (int16 max >= thr -> re-score)
   OvfRec* ovf;
   int* ovf_count;
   int ovf_cap;
-  int qidx;
   uint32_t code_pad2;        // PAD | PAD << 8
   uint32_t nGe, nGsGe;       // packed s16x2 -Ge, -(Gs+Ge)
 };
@@ -83,7 +90,7 @@ struct RescoreArgs {
   int alpha;
   const OvfRec* ovf;
   const int* ovf_count;
-  int2* bbuf;                // [gridDim*warps][bcap]
+  int2* bbuf;                // link rows, [gridDim][RESCORE_WARPS][bcap]
   int bcap;
   int32_t* scores;           // [nq][n_seqs]
   int64_t n_seqs;
@@ -97,7 +104,7 @@ int inter_max_ctas_per_sm(int G, int R, int NT, int smem_bytes);
 cudaError_t launch_inter(int G, int R, int NT, int grid, int smem_bytes, const InterArgs& a, cudaStream_t st);
 bool inter_config_supported(int G, int R);
 cudaError_t launch_rescore(int grid, const RescoreArgs& a, cudaStream_t st);
-constexpr int RESCORE_WARPS = 4;
+constexpr int RESCORE_WARPS = 8;
 constexpr int RESCORE_R = 8;
 
 }  // namespace swdual

@@ -10,7 +10,8 @@ import paper_conf_icpp_kedad_sidhoummmmt14_b200 as sw  # noqa: E402
 
 m = int(os.environ.get("PROF_M", "567"))
 reps = int(os.environ.get("PROF_REPS", "2"))
-c = swgen.make_config("c2", n_db=int(os.environ.get("PROF_NDB", "570000")))
+wl = os.environ.get("PROF_WORKLOAD", "c2")
+c = swgen.make_config(wl, n_db=int(os.environ["PROF_NDB"]) if os.environ.get("PROF_NDB") else None)
 h = sw.Handle(0)
 for k in ("force_G", "force_R"):
     if os.environ.get(k.upper()):

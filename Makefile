@@ -22,7 +22,7 @@ $(OBJ)/%.o: $(SRC)/%.cpp $(HDRS)
 	$(NVCC) $(NVFLAGS) -c $< -o $@
 
 $(LIB): $(OBJS)
-	$(NVCC) $(ARCH) -shared -o $@.tmp $(OBJS) && mv $@.tmp $@
+	$(NVCC) $(ARCH) -shared -Xlinker --no-undefined -o $@.tmp $(OBJS) -lcudart_static -lrt -lpthread -ldl && mv $@.tmp $@
 
 clean:
 	rm -rf build $(LIB)

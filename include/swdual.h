@@ -124,6 +124,8 @@ int32_t sw_last_stats(sw_handle_t h, sw_stats_t* out);
  * Integer options (testing / tuning).  Keys:
  *   "overflow_threshold"  force the int16 re-score threshold (0 = automatic)
  *   "force_G", "force_R"  force the inter-task lane-group geometry (0 = auto)
+ *   "query_pairs"         1 (default): queries are paired two per s16x2 register for
+ *                         the short DB pairs (no PRMT); 0: one query per register
  *   "t_long"              DB pairs longer than this (default 3000) are scored in
  *                         the intra-task mode (all warps of a CTA on one pair);
  *                         applies to databases loaded afterwards

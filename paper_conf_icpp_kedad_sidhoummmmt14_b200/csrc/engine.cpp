@@ -92,6 +92,7 @@ struct sw_handle_s {
   // options
   int64_t opt_thr = 0, opt_G = 0, opt_R = 0;
   int64_t opt_t_long = T_LONG;  // pairs longer than this use the intra-task (long) mode
+  int64_t opt_query_pairs = 1;  // pair queries two per register for the short pairs
   // last-search bookkeeping
   sw_stats_t stats{};
   cudaStream_t last_stream = nullptr;
@@ -150,7 +151,8 @@ static ProfGeom make_geom(int G, int R, int m, int alpha) {
 // (row padding to whole strips, wavefront fill of G-1 columns per pair and
 // strip, a per-step overhead amortised over R rows, a register-pressure
 // penalty for the largest R).
-static void choose_geom(const sw_handle_s* h, const std::vector<int>& ms, double Lavg, int& G, int& R) {
+static void choose_geom(const sw_handle_s* h, const std::vector<std::pair<int, int>>& slots, double Lavg, int& G,
+                        int& R) {
   if (h->opt_G > 0 && h->opt_R > 0) {
     G = int(h->opt_G);
     R = int(h->opt_R);
@@ -165,10 +167,12 @@ static void choose_geom(const sw_handle_s* h, const std::vector<int>& ms, double
     for (int r : Rs) {
       const double per_cell = 1.0 + 7.0 / (5.5 * r) + (r > 24 ? 0.06 : 0.0);
       double cost = 0;
-      for (int m : ms) {
+      for (auto [m, mode] : slots) {
         const int strips = std::max(1, (m + g * r - 1) / (g * r));
         const double rows = double(strips) * g * r;
-        cost += rows * (Lavg + g) * per_cell * (strips > 1 ? 1.02 : 1.0);
+        // mode 1 (query pair) sweeps every DB sequence once for two queries, without the PRMT
+        const double cols = mode == 1 ? 2.0 * (Lavg + g) * (5.5 / 6.5) : (Lavg + g);
+        cost += rows * cols * per_cell * (strips > 1 ? 1.02 : 1.0);
       }
       if (cost < best) { best = cost; G = g; R = r; }
     }
@@ -215,6 +219,8 @@ int32_t sw_set_option(sw_handle_t h, const char* key, int64_t value) {
   } else if (k == "t_long") {
     if (value < 0) return set_err(h, SW_EINVAL, "t_long must be >= 0");
     h->opt_t_long = value;
+  } else if (k == "query_pairs") {
+    h->opt_query_pairs = value;
   } else if (k == "timing_accumulate") {
     h->timing_accumulate = value != 0;  // keep kernel events across searches until "timing_reset"
     h->n_events_used = 0;
@@ -325,24 +331,45 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
   std::stable_sort(order.begin(), order.end(), [&](int x, int y) { return qlen[size_t(x)] > qlen[size_t(y)]; });
   std::vector<int> ms;
   for (int i : order) ms.push_back(int(qlen[size_t(i)]));
+  // short-pair slots: neighbours in length order form query pairs (mode 1)
+  struct Slot { int mode, k0, k1; };
+  std::vector<Slot> slots;
+  const bool pairs_on = h->opt_query_pairs != 0;
+  for (size_t k = 0; k < order.size();) {
+    if (pairs_on && k + 1 < order.size()) { slots.push_back({1, int(k), int(k + 1)}); k += 2; }
+    else { slots.push_back({0, int(k), -1}); k += 1; }
+  }
+  std::vector<std::pair<int, int>> slot_m;
+  for (auto& sl : slots) slot_m.push_back({ms[size_t(sl.k0)], sl.mode});
   int G = 4, R = 24;
-  choose_geom(h, ms, nshort > 0 ? c.sum_short / nshort : 1.0, G, R);
+  choose_geom(h, slot_m, nshort > 0 ? c.sum_short / nshort : 1.0, G, R);
   if (!inter_config_supported(G, R)) fail(SW_EUNSUPPORTED, "no kernel for this geometry");
   const int NT = 256, NG = NT / G, W = NT / 32;
-  // profiles: short (G x R) and long (32 x LONG_R) geometry for every query
+  const int LB2 = (((R / 4) | 1) * 16);
+  const int LS2 = G * LB2;
+  const int SB2 = (((alpha + 1) * LS2 + 15) / 16) * 16;
+  // profiles: long geometry per query; short geometry per slot
   size_t total = 0;
-  std::vector<ProfGeom> gs, gl;
-  std::vector<size_t> off_s, off_l;
+  std::vector<ProfGeom> gl;
+  std::vector<size_t> off_l;
   for (int m : ms) {
-    gs.push_back(make_geom(G, R, m, alpha));
     gl.push_back(make_geom(32, LONG_R, m, alpha));
-    off_s.push_back(total);
-    total += nshort > 0 ? size_t(gs.back().n_strips) * gs.back().SB : 0;
     off_l.push_back(total);
     total += nlong > 0 ? size_t(gl.back().n_strips) * gl.back().SB : 0;
   }
+  const ProfGeom g1 = make_geom(G, R, 1, alpha);  // SB / LS / LB of the mode-0 profile
+  std::vector<size_t> off_s;
+  std::vector<int> strips_s;
+  for (auto& sl : slots) {
+    const int n = std::max(1, (ms[size_t(sl.k0)] + G * R - 1) / (G * R));  // k0 is the longer query
+    strips_s.push_back(n);
+    off_s.push_back(total);
+    if (nshort > 0) total += size_t(n) * (sl.mode == 1 ? SB2 : g1.SB);
+  }
   SW_CK(h->prof.ensure(total + 16));
   uint8_t* prof = h->prof.as<uint8_t>();
+  const int8_t* dmat = h->matrix.as<int8_t>();
+  auto qptr = [&](int k) { return h->qcodes.as<uint8_t>() + qoff0[size_t(order[size_t(k)])]; };
   std::vector<QueryDesc> desc(order.size());
   double sumS = 0, sumL = 0;
   for (int p = 0; p < np; ++p) {
@@ -351,32 +378,61 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
   }
   for (size_t k = 0; k < order.size(); ++k) {
     const int qi = order[k];
-    const uint8_t* dq = h->qcodes.as<uint8_t>() + qoff0[size_t(qi)];
-    if (nshort > 0) {
-      SW_CK(launch_build_profile(dq, ms[k], h->matrix.as<int8_t>(), alpha, gs[k], prof + off_s[k], c.st));
-      ++launches;
-    }
     if (nlong > 0) {
-      SW_CK(launch_build_profile(dq, ms[k], h->matrix.as<int8_t>(), alpha, gl[k], prof + off_l[k], c.st));
+      SW_CK(launch_build_profile(qptr(int(k)), ms[k], dmat, alpha, gl[k], prof + off_l[k], c.st));
       ++launches;
     }
     QueryDesc& d = desc[k];
-    d.prof = prof + off_s[k];
+    d.prof = nullptr;
     d.prof_long = prof + off_l[k];
     d.scores = c.dscores + int64_t(qi) * db->n_seqs;
-    d.n_strips = gs[k].n_strips;
+    d.n_strips = 0;
     d.n_strips_long = gl[k].n_strips;
     d.qidx = qi;
     d.pad_ = 0;
-    cells_computed += 2.0 * sumS * double(gs[k].n_strips) * G * R + 2.0 * sumL * double(gl[k].n_strips) * 32 * LONG_R;
+    cells_computed += 2.0 * sumL * double(gl[k].n_strips) * 32 * LONG_R;
   }
-  SW_CK(h->qdesc.ensure(desc.size() * sizeof(QueryDesc)));
-  SW_CK(cudaMemcpyAsync(h->qdesc.p, desc.data(), desc.size() * sizeof(QueryDesc), cudaMemcpyHostToDevice, c.st));
-  const ProfGeom g0 = gs[0], l0 = gl[0];
-  const int smem = g0.SB + (nlong > 0 ? W * l0.SB : 0);
+  std::vector<SlotDesc> sdesc(slots.size());
+  int item = 0;
+  for (size_t j = 0; j < slots.size(); ++j) {
+    const Slot& sl = slots[j];
+    SlotDesc& d = sdesc[j];
+    d.prof = prof + off_s[j];
+    d.mode = sl.mode;
+    d.n_strips = strips_s[j];
+    d.qidx0 = order[size_t(sl.k0)];
+    d.scores0 = c.dscores + int64_t(d.qidx0) * db->n_seqs;
+    d.qidx1 = sl.mode == 1 ? order[size_t(sl.k1)] : -1;
+    d.scores1 = sl.mode == 1 ? c.dscores + int64_t(d.qidx1) * db->n_seqs : nullptr;
+    d.item_begin = item;
+    d.n_items = nshort > 0 ? (sl.mode == 1 ? (2 * nshort + NG - 1) / NG : (nshort + NG - 1) / NG) : 0;
+    item += d.n_items;
+    if (nshort > 0) {
+      if (sl.mode == 1) {
+        SW_CK(launch_build_profile_q2(qptr(sl.k0), ms[size_t(sl.k0)], qptr(sl.k1), ms[size_t(sl.k1)], dmat, alpha,
+                                      G, R, LB2, d.n_strips, SB2, prof + off_s[j], c.st));
+        cells_computed += 2.0 * (2.0 * sumS) * double(d.n_strips) * G * R;  // every sequence, 2 queries
+      } else {
+        ProfGeom gq = g1;
+        gq.n_strips = d.n_strips;
+        SW_CK(launch_build_profile(qptr(sl.k0), ms[size_t(sl.k0)], dmat, alpha, gq, prof + off_s[j], c.st));
+        cells_computed += 2.0 * sumS * double(d.n_strips) * G * R;
+      }
+      ++launches;
+    }
+  }
+  SW_CK(h->qdesc.ensure(desc.size() * sizeof(QueryDesc) + sdesc.size() * sizeof(SlotDesc) + 16));
+  QueryDesc* d_desc = h->qdesc.as<QueryDesc>();
+  SlotDesc* d_slots = reinterpret_cast<SlotDesc*>(d_desc + desc.size());
+  SW_CK(cudaMemcpyAsync(d_desc, desc.data(), desc.size() * sizeof(QueryDesc), cudaMemcpyHostToDevice, c.st));
+  SW_CK(cudaMemcpyAsync(d_slots, sdesc.data(), sdesc.size() * sizeof(SlotDesc), cudaMemcpyHostToDevice, c.st));
+  std::vector<ProfGeom> gs;
+  for (size_t j = 0; j < slots.size(); ++j) { ProfGeom x = g1; x.n_strips = strips_s[j]; gs.push_back(x); }
+  const ProfGeom g0 = g1, l0 = gl[0];
+  const int smem = std::max(g0.SB, SB2) + (nlong > 0 ? W * l0.SB : 0);
   const int occ = inter_max_ctas_per_sm(G, R, NT, smem);
   if (occ <= 0) fail(SW_ECUDA, "inter kernel does not fit on an SM");
-  const int64_t n_items = int64_t(order.size()) * (nlong + (nshort + NG - 1) / NG);
+  const int64_t n_items = int64_t(order.size()) * nlong + item;
   if (n_items >= (int64_t(1) << 31)) fail(SW_EUNSUPPORTED, "too many work items");
   const int grid = int(std::max<int64_t>(1, std::min<int64_t>(n_items, int64_t(occ) * h->sms)));
   int max_strips = 1;
@@ -390,8 +446,14 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
   SW_CK(h->counters.ensure(sizeof(int)));
   SW_CK(cudaMemsetAsync(h->counters.p, 0, sizeof(int), c.st));
   InterArgs a{};
-  a.queries = h->qdesc.as<QueryDesc>();
+  a.queries = d_desc;
   a.n_queries = int(order.size());
+  a.slots = d_slots;
+  a.n_slots = int(slots.size());
+  a.n_short_items = item;
+  a.SB2 = SB2;
+  a.LS2 = LS2;
+  a.LB2 = LB2;
   a.SB = g0.SB;
   a.LS = g0.LS;
   a.LB = g0.LB;

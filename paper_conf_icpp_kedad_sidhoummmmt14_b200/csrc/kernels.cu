@@ -64,6 +64,46 @@ cudaError_t launch_build_profile(const uint8_t* q, int m, const int8_t* matrix, 
   return cudaGetLastError();
 }
 
+// Query-pair profile: 32-bit word per (strip, letter, lane, row):
+//   low 16 = S[qa[row]][a], high 16 = S[qb[row]][a]  (PAD rows / letters: PAD_SCORE)
+__global__ void build_profile_q2_kernel(const uint8_t* __restrict__ qa, int ma, const uint8_t* __restrict__ qb,
+                                        int mb, const int8_t* __restrict__ M, int alpha, int G, int R, int LB2,
+                                        int n_strips, int SB2, uint32_t* __restrict__ prof) {
+  const int LS2 = G * LB2;
+  const int64_t total = (int64_t)n_strips * (SB2 / 4);
+  for (int64_t i = blockIdx.x * (int64_t)blockDim.x + threadIdx.x; i < total;
+       i += (int64_t)gridDim.x * blockDim.x) {
+    const int s = int(i / (SB2 / 4));
+    const int rem = int(i - (int64_t)s * (SB2 / 4)) * 4;  // byte offset within the strip
+    uint32_t v = 0;
+    if (rem < (alpha + 1) * LS2) {
+      const int a = rem / LS2;
+      const int rr = rem - a * LS2;
+      const int k = rr / LB2;
+      const int r = (rr - k * LB2) / 4;
+      if (r < R) {
+        const int row = s * G * R + k * R + r;
+        const int va = (row < ma && a < alpha) ? M[qa[row] * alpha + a] : PAD_SCORE;
+        const int vb = (row < mb && a < alpha) ? M[qb[row] * alpha + a] : PAD_SCORE;
+        v = (uint32_t(va) & 0xffffu) | (uint32_t(vb) << 16);
+      }
+    }
+    prof[i] = v;
+  }
+}
+
+cudaError_t launch_build_profile_q2(const uint8_t* qa, int ma, const uint8_t* qb, int mb, const int8_t* matrix,
+                                    int alpha, int G, int R, int LB2, int n_strips, int SB2, uint8_t* prof,
+                                    cudaStream_t st) {
+  const int64_t total = (int64_t)n_strips * (SB2 / 4);
+  int grid = int((total + 255) / 256);
+  if (grid > 4096) grid = 4096;
+  if (grid < 1) grid = 1;
+  build_profile_q2_kernel<<<grid, 256, 0, st>>>(qa, ma, qb, mb, matrix, alpha, G, R, LB2, n_strips, SB2,
+                                                reinterpret_cast<uint32_t*>(prof));
+  return cudaGetLastError();
+}
+
 // Warp-uniform wait until a shared progress counter reaches `need` (all lanes
 // read the broadcast word; __all_sync keeps the warp converged so the shuffles
 // that follow stay on the fast path), then a CTA-scope acquire fence.
@@ -89,12 +129,12 @@ __device__ __forceinline__ void copy_strip(uint8_t* dst, const uint8_t* __restri
 // strip's bottom row at wp[t] (t = step).  LINKED: the row above is produced
 // concurrently by another warp of the CTA (intra-task mode): lane 0 waits on
 // its progress counter, lane G-1 publishes its own.
-template <int G, int R, bool LINKED>
+template <int G, int R, bool LINKED, bool Q2 = false>
 __device__ __forceinline__ void strip_pass(const uint8_t* sprof, int LS, int LB, const uint16_t* pstream, int L,
                                            int T, int k, bool rd, bool wr, const uint2* __restrict__ rp,
                                            uint2* __restrict__ wp, volatile int* prog_in, int need_base,
                                            volatile int* prog_out, int pub_base, uint32_t code_pad2, uint32_t nGe,
-                                           uint32_t nGsGe, uint32_t& best) {
+                                           uint32_t nGsGe, uint32_t& best, uint32_t shift = 0) {
   uint32_t Hl[R], E[R];
 #pragma unroll
   for (int r = 0; r < R; ++r) { Hl[r] = 0; E[r] = 0; }
@@ -148,9 +188,15 @@ __device__ __forceinline__ void strip_pass(const uint8_t* sprof, int LS, int LB,
         rH = tv.x;
         rF = tv.y;
       }
-      const uint8_t* pa = sprof + (rC & 0xffu) * LS + laneoff;
-      const uint8_t* pb = sprof + (rC >> 8) * LS + laneoff;
-      gotoh_column<R>(Hl, E, best, hdiag, pa, pb, rH, rF, nGe, nGsGe);
+      if constexpr (Q2) {
+        // one DB sequence (byte `shift` of the pair word) against two queries
+        const uint8_t* pa = sprof + ((rC >> shift) & 0xffu) * LS + laneoff;
+        gotoh_column_q2<R>(Hl, E, best, hdiag, pa, rH, rF, nGe, nGsGe);
+      } else {
+        const uint8_t* pa = sprof + (rC & 0xffu) * LS + laneoff;
+        const uint8_t* pb = sprof + (rC >> 8) * LS + laneoff;
+        gotoh_column<R>(Hl, E, best, hdiag, pa, pb, rH, rF, nGe, nGsGe);
+      }
       sH = rH;
       sF = rF;
       sC = rC;
@@ -200,8 +246,8 @@ __device__ __forceinline__ void emit_pair(const InterArgs& a, const QueryDesc& d
 template <int G, int R, int NT>
 __global__ void __launch_bounds__(NT) inter_kernel(InterArgs a) {
   extern __shared__ __align__(16) uint8_t smem[];
-  uint8_t* sprof = smem;           // short-mode strip profile (a.SB bytes)
-  uint8_t* lprof = smem + a.SB;    // long mode: one a.SBL slot per warp
+  uint8_t* sprof = smem;                         // short-mode strip profile (max(SB, SB2) bytes)
+  uint8_t* lprof = smem + max(a.SB, a.SB2);      // long mode: one a.SBL slot per warp
   __shared__ int s_item;
   __shared__ int s_prog[NT / 32];
   __shared__ uint32_t s_best[NT / 32];
@@ -211,10 +257,8 @@ __global__ void __launch_bounds__(NT) inter_kernel(InterArgs a) {
   const int k = tid & (G - 1);
   const int g = tid / G;
   const int lane = tid & 31, warp = tid >> 5;
-  const int n_short = a.pair_end - a.pair_begin;
-  const int nchunks = (n_short + NG - 1) / NG;
   const int n_long_items = a.n_queries * a.n_long;
-  const int n_items = n_long_items + a.n_queries * nchunks;
+  const int n_items = n_long_items + a.n_short_items;
   uint2* __restrict__ bb = a.bbuf + ((size_t)blockIdx.x * NG + g) * (size_t)a.bcap;
   int loaded = -1;  // (query rank << 16 | strip) of the short profile in shared memory (CTA-uniform)
 
@@ -258,32 +302,73 @@ __global__ void __launch_bounds__(NT) inter_kernel(InterArgs a) {
         emit_pair(a, d, pidx, pr, b);
       }
     } else {
-      // ---------------- chunk of short pairs, one per lane group
+      // ---------------- short work: find the slot of this item (slots are few)
       const int c = item - n_long_items;
-      const int qr = c / nchunks, chunk = c - qr * nchunks;
-      const QueryDesc d = a.queries[qr];
-      const int p = a.pair_begin + chunk * NG + g;
-      const bool valid = p < a.pair_end;
+      int lo = 0, hi = a.n_slots - 1;
+      while (lo < hi) {
+        const int mid = (lo + hi + 1) >> 1;
+        if (a.slots[mid].item_begin <= c) lo = mid; else hi = mid - 1;
+      }
+      const int sl = lo;
+      const SlotDesc d = a.slots[sl];
+      const int chunk = c - d.item_begin;
+      const bool q2 = d.mode == 1;
+      int p, half = 0;
+      if (q2) {  // chunk of NG half-pairs: DB sequence = one half of a pair
+        const int hp = chunk * NG + g;
+        p = a.pair_begin + (hp >> 1);
+        half = hp & 1;
+      } else {
+        p = a.pair_begin + chunk * NG + g;
+      }
+      bool valid = p < a.pair_end;
       PairRec pr;
       if (valid) pr = a.pairs[p];
       else { pr.off = 0; pr.len = 0; pr.id0 = -1; pr.id1 = -1; }
+      if (q2 && half && pr.id1 < 0) valid = false;  // odd leftover pair has no high half
       int T = pr.len + G;                          // lane G-1 finishes column len-1 at step len+G-2
       if (G < 32) T = __reduce_max_sync(FULL, T);  // warp-uniform trip count (shuffles)
       uint32_t best = 0;
+      const int SBx = q2 ? a.SB2 : a.SB;
       for (int s = 0; s < d.n_strips; ++s) {
-        const int want = (qr << 16) | s;
+        const int want = (sl << 16) | s;
         if (want != loaded) {
           __syncthreads();
-          copy_strip(sprof, d.prof + (size_t)s * a.SB, a.SB);
+          copy_strip(sprof, d.prof + (size_t)s * SBx, SBx);
           __syncthreads();
           loaded = want;
         }
-        strip_pass<G, R, false>(sprof, a.LS, a.LB, a.stream + pr.off, pr.len, T, k, s > 0, s + 1 < d.n_strips,
-                                bb + (G - 1), bb, nullptr, 0, nullptr, 0, a.code_pad2, a.nGe, a.nGsGe, best);
+        if (q2)
+          strip_pass<G, R, false, true>(sprof, a.LS2, a.LB2, a.stream + pr.off, pr.len, T, k, s > 0,
+                                        s + 1 < d.n_strips, bb + (G - 1), bb, nullptr, 0, nullptr, 0, a.code_pad2,
+                                        a.nGe, a.nGsGe, best, half ? 8u : 0u);
+        else
+          strip_pass<G, R, false>(sprof, a.LS, a.LB, a.stream + pr.off, pr.len, T, k, s > 0, s + 1 < d.n_strips,
+                                  bb + (G - 1), bb, nullptr, 0, nullptr, 0, a.code_pad2, a.nGe, a.nGsGe, best);
       }
 #pragma unroll
       for (int o = G / 2; o > 0; o >>= 1) best = __vmaxs2(best, __shfl_xor_sync(FULL, best, o, G));
-      if (valid && k == 0) emit_pair(a, d, p, pr, best);
+      if (valid && k == 0) {
+        if (q2) {
+          const int id = half ? pr.id1 : pr.id0;
+          const int v0 = int(int16_t(best & 0xffffu)), v1 = int(int16_t(best >> 16));
+          d.scores0[id] = v0;
+          d.scores1[id] = v1;
+          if (v0 >= a.thr) {
+            const int e = atomicAdd(a.ovf_count, 1);
+            if (e < a.ovf_cap) a.ovf[e] = OvfRec{d.qidx0, p, half, 0};
+          }
+          if (v1 >= a.thr) {
+            const int e = atomicAdd(a.ovf_count, 1);
+            if (e < a.ovf_cap) a.ovf[e] = OvfRec{d.qidx1, p, half, 0};
+          }
+        } else {
+          QueryDesc qd;
+          qd.scores = d.scores0;
+          qd.qidx = d.qidx0;
+          emit_pair(a, qd, p, pr, best);
+        }
+      }
     }
     __syncthreads();
   }
@@ -336,9 +421,10 @@ cudaError_t launch_inter(int G, int R, int NT, int grid, int smem_bytes, const I
 // ---------------------------------------------------------------------------
 // Exact int32 re-score of flagged pairs.  One CTA per pair,
 // the same chained-warp intra-task wavefront as the long-pair mode but one
-// problem per lane in int32 and S read from a shared 33x33 matrix: warp w does
-// strips w, w+W, ... (32 lanes x RESCORE_R rows), strip s+1 consuming strip s's
-// bottom row through a global link row + shared progress counter.
+// problem per lane in int32 (s32 DPX) and S read from a shared 33x33 matrix:
+// warp w does strips w, w+W, ... (32 lanes x RESCORE_R rows), strip s+1
+// consuming strip s's bottom row through a global link row + shared progress
+// counter.  Codes and link cells are fetched a 4-column block ahead.
 __global__ void __launch_bounds__(RESCORE_WARPS * 32) rescore_kernel(RescoreArgs a) {
   constexpr int R = RESCORE_R;
   constexpr int W = RESCORE_WARPS;
@@ -351,9 +437,11 @@ __global__ void __launch_bounds__(RESCORE_WARPS * 32) rescore_kernel(RescoreArgs
     sm[i] = (x < a.alpha && y < a.alpha) ? int(a.matrix[x * a.alpha + y]) : int(PAD_SCORE);
   }
   const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
+  const bool lead = lane == 0, tail = lane == 31;
   int2* __restrict__ links = a.bbuf + (size_t)blockIdx.x * W * a.bcap;
   const int cnt = *a.ovf_count;
   const int pad = a.alpha;
+  const int nGe = -a.Ge, nGsGe = -(a.Gs + a.Ge);
   for (int e = blockIdx.x; e < cnt; e += gridDim.x) {
     __syncthreads();
     if (threadIdx.x < W) { s_prog[threadIdx.x] = -1; s_best[threadIdx.x] = 0; }
@@ -363,15 +451,17 @@ __global__ void __launch_bounds__(RESCORE_WARPS * 32) rescore_kernel(RescoreArgs
     const uint8_t* qc = a.qcodes + a.qoff[o.q];
     const int m = int(a.qoff[o.q + 1] - a.qoff[o.q]);
     const int L = pr.len;
-    const int shift = o.half ? 8 : 0;
+    const uint32_t shift = o.half ? 8u : 0u;
     const int nstrips = (m + 32 * R - 1) / (32 * R);
     const int T = L + 32;
+    const uint2* __restrict__ codes = reinterpret_cast<const uint2*>(a.stream + pr.off);
+    const uint32_t padw = uint32_t(pad) * 0x01010101u;
     int best = 0;
     for (int s = warp; s < nstrips; s += W) {
       const bool rd = s > 0, wr = s + 1 < nstrips;
       const int lin = (s + W - 1) % W, lout = s % W;
-      const int2* rp = links + (size_t)lin * a.bcap + 31;
-      int2* wp = links + (size_t)lout * a.bcap;
+      const int2* __restrict__ rp = links + (size_t)lin * a.bcap + 31;
+      int2* __restrict__ wp = links + (size_t)lout * a.bcap;
       volatile int* pin = &s_prog[lin];
       volatile int* pout = &s_prog[lout];
       const int need_base = (s - 1) << 20, pub_base = s << 20;
@@ -384,47 +474,67 @@ __global__ void __launch_bounds__(RESCORE_WARPS * 32) rescore_kernel(RescoreArgs
         E[r] = 0;
       }
       int hdiag = 0, sH = 0, sF = 0, sC = pad;
-      for (int t = 0; t < T; ++t) {
-        int rH = __shfl_up_sync(FULL, sH, 1);
-        int rF = __shfl_up_sync(FULL, sF, 1);
-        int rC = __shfl_up_sync(FULL, sC, 1);
-        if (rd && t < L && (t & 3) == 0) wait_progress(pin, need_base + min(t + 36 + LINK_LAG, L + 32));
-        if (lane == 0) {
-          if (t < L) {
-            rC = (a.stream[pr.off + t] >> shift) & 0xff;
-            if (rd) {
-              const int2 v = __ldcg(rp + t);
-              rH = v.x;
-              rF = v.y;
-            } else { rH = 0; rF = 0; }
-          } else { rC = pad; rH = 0; rF = 0; }
-        }
-        __syncwarp();
-        int hd = hdiag;
-        hdiag = rH;
-        int F = rF;
-#pragma unroll
-        for (int r = 0; r < R; ++r) {
-          const int h = max(max(hd + sm[qr[r] + rC], E[r]), F);        // Eq. (2) (E, F >= 0)
-          hd = Hl[r];
-          Hl[r] = h;
-          const int tt = h - a.Gs - a.Ge;
-          E[r] = max(max(E[r] - a.Ge, tt), 0);                          // Eq. (3)
-          F = max(max(F - a.Ge, tt), 0);                                // Eq. (4)
-          best = max(best, h);
-        }
-        sH = Hl[R - 1];
-        sF = F;
-        sC = rC;
-        if (wr && lane == 31) __stcg(wp + t, make_int2(sH, sF));
-        if (wr && (t & 3) == 3) {
-          __syncwarp();
-          if (lane == 31) { __threadfence_block(); *pout = pub_base + t + 1; }
-        }
+      const int2 z2 = make_int2(0, 0);
+      uint2 cw = make_uint2(padw, padw);
+      int2 tb0 = z2, tb1 = z2, tb2 = z2, tb3 = z2;
+      if (rd && L > 0) wait_progress(pin, need_base + min(4 + 31 + LINK_LAG, L + 32));
+      if (lead && L > 0) {
+        cw = codes[0];
+        if (rd) { tb0 = __ldcg(rp + 0); tb1 = __ldcg(rp + 1); tb2 = __ldcg(rp + 2); tb3 = __ldcg(rp + 3); }
       }
-      if (wr) {
+      __syncwarp();
+      for (int t0 = 0; t0 < T; t0 += 4) {
+        const uint2 cwc = cw;
+        const int2 c0 = tb0, c1 = tb1, c2 = tb2, c3 = tb3;
+        if (rd && t0 + 4 < L) wait_progress(pin, need_base + min(t0 + 8 + 31 + LINK_LAG, L + 32));
+        if (lead) {
+          if (t0 + 4 < L) {
+            cw = codes[(t0 + 4) >> 2];
+            if (rd) {
+              tb0 = __ldcg(rp + t0 + 4); tb1 = __ldcg(rp + t0 + 5); tb2 = __ldcg(rp + t0 + 6); tb3 = __ldcg(rp + t0 + 7);
+            }
+          } else {
+            cw = make_uint2(padw, padw);
+            tb0 = z2; tb1 = z2; tb2 = z2; tb3 = z2;
+          }
+        }
         __syncwarp();
-        if (lane == 31) { __threadfence_block(); *pout = pub_base + T; }
+#pragma unroll
+        for (int j = 0; j < 4; ++j) {
+          int rH = __shfl_up_sync(FULL, sH, 1);
+          int rF = __shfl_up_sync(FULL, sF, 1);
+          int rC = __shfl_up_sync(FULL, sC, 1);
+          if (lead) {
+            const uint32_t w = (j < 2) ? cwc.x : cwc.y;
+            rC = int(((j & 1) ? (w >> 16) : w) >> shift) & 0xff;
+            const int2 tv = (j == 0) ? c0 : (j == 1) ? c1 : (j == 2) ? c2 : c3;
+            rH = tv.x;
+            rF = tv.y;
+          }
+          int hd = hdiag;
+          hdiag = rH;
+          int F = rF;
+          int hprev = 0;
+#pragma unroll
+          for (int r = 0; r < R; ++r) {
+            const int h = max(__viaddmax_s32(hd, sm[qr[r] + rC], E[r]), F);  // Eq. (2) (E, F >= 0)
+            hd = Hl[r];
+            Hl[r] = h;
+            const int tt = h + nGsGe;
+            E[r] = __viaddmax_s32_relu(E[r], nGe, tt);                               // Eq. (3)
+            F = __viaddmax_s32_relu(F, nGe, tt);                                     // Eq. (4)
+            if (r & 1) best = __vimax3_s32(best, hprev, h);
+            else hprev = h;
+          }
+          sH = Hl[R - 1];
+          sF = F;
+          sC = rC;
+          if (wr && tail) __stcg(wp + t0 + j, make_int2(sH, sF));
+        }
+        if (wr) {
+          __syncwarp();
+          if (tail) { __threadfence_block(); *pout = pub_base + t0 + 4; }
+        }
       }
     }
 #pragma unroll

@@ -59,10 +59,28 @@ struct QueryDesc {
   int qidx, pad_;
 };
 
+// Short-pair work of one "slot": a single query (mode 0: two DB sequences per
+// s16x2 register, int8 profile) or a query PAIR (mode 1: two queries per
+// register, one DB sequence per lane group, s16x2 profile).
+struct SlotDesc {
+  const uint8_t* prof;       // mode 0: [n_strips][SB] int8; mode 1: [n_strips][SB2] s16x2
+  int32_t* scores0;          // scores row of the (first) query
+  int32_t* scores1;          // mode 1: row of the second query
+  int n_strips;
+  int mode;
+  int qidx0, qidx1;
+  int item_begin;            // first short work item of this slot
+  int n_items;               // short work items of this slot
+};
+
 struct InterArgs {
-  const QueryDesc* queries;  // [n_queries], processing order
+  const QueryDesc* queries;  // [n_queries], processing order (long items)
   int n_queries;
-  int SB, LS, LB;            // short geometry (G, R of the launch)
+  const SlotDesc* slots;     // [n_slots] short-pair work
+  int n_slots;
+  int n_short_items;         // sum of slots' n_items
+  int SB, LS, LB;            // short geometry (G, R of the launch), mode 0 profile
+  int SB2, LS2, LB2;         // mode 1 (query-pair) profile
   int SBL, LSL, LBL;         // long geometry (32 lanes x LONG_R rows)
   int n_long;                // pairs [0, n_long) are long (intra-task items)
   uint2* links;              // [gridDim][NT/32][lcap] strip-to-strip rows (long items)
@@ -100,11 +118,15 @@ struct RescoreArgs {
 // kernels.cu entry points (host side launchers); return cudaError_t
 cudaError_t launch_build_profile(const uint8_t* q, int m, const int8_t* matrix, int alpha,
                                  const ProfGeom& g, uint8_t* prof, cudaStream_t st);
+// query-pair profile: word = S[qa_i][a] (low 16) | S[qb_i][a] << 16, lane block LB2
+cudaError_t launch_build_profile_q2(const uint8_t* qa, int ma, const uint8_t* qb, int mb, const int8_t* matrix,
+                                    int alpha, int G, int R, int LB2, int n_strips, int SB2, uint8_t* prof,
+                                    cudaStream_t st);
 int inter_max_ctas_per_sm(int G, int R, int NT, int smem_bytes);
 cudaError_t launch_inter(int G, int R, int NT, int grid, int smem_bytes, const InterArgs& a, cudaStream_t st);
 bool inter_config_supported(int G, int R);
 cudaError_t launch_rescore(int grid, const RescoreArgs& a, cudaStream_t st);
-constexpr int RESCORE_WARPS = 8;
+constexpr int RESCORE_WARPS = 16;
 constexpr int RESCORE_R = 8;
 
 }  // namespace swdual

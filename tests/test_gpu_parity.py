@@ -228,3 +228,14 @@ def test_config_c4_sampled():
     ref = oracle_scores(c["qcodes"], c["qoff"], sub, sub_off, procs=16)
     assert ref.max() > 32767  # planted self-hits of >= 6.4k queries really overflow int16
     np.testing.assert_array_equal(got[:, idx], ref)
+
+
+@pytest.mark.parametrize("pairs", [0, 1])
+def test_query_pairing_modes(pairs):
+    """Two queries per register (mode 1) and one (mode 0), odd query counts,
+    very unequal pair lengths (the shorter query padded with PAD rows)."""
+    rng = np.random.default_rng(31 + pairs)
+    dc, do = _seqs(list(rng.integers(1, 600, size=150)) + [0, 1, 2, 3], rng)
+    qc, qo = _seqs([700, 31, 256, 255, 1, 90, 400], rng)
+    got = gpu_scores(qc, qo, dc, do, opts={"query_pairs": pairs})
+    np.testing.assert_array_equal(got, oracle_scores(qc, qo, dc, do))

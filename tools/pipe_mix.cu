@@ -43,6 +43,20 @@ __global__ void k_mix(uint32_t* out, uint32_t seed) {
         a[i] = __viaddmax_s16x2_relu(a[i], k1, c[i]);
         asm volatile("max.s16x2 %0, %0, %1;" : "+r"(b[i]) : "r"(c[i]));
         c[i] += 0x00010001u;
+      } else if constexpr (MIX == 8) {   // 1 HMNMX2 (max.f16x2)
+        asm volatile("max.f16x2 %0, %0, %1;" : "+r"(a[i]) : "r"(c[i]));
+        c[i] += 0x00010001u;
+      } else if constexpr (MIX == 9) {   // VIADDMNMX + HMNMX2 (independent)
+        a[i] = __viaddmax_s16x2_relu(a[i], k1, c[i]);
+        asm volatile("max.f16x2 %0, %0, %1;" : "+r"(b[i]) : "r"(c[i]));
+      } else if constexpr (MIX == 10) {  // VIADD.16x2 + HMNMX2 (independent)
+        a[i] = __vadd2(a[i], k1);
+        asm volatile("max.f16x2 %0, %0, %1;" : "+r"(b[i]) : "r"(c[i]));
+      } else if constexpr (MIX == 11) {  // 2 VIADDMNMX + VIADD.16x2 + HMNMX2
+        a[i] = __viaddmax_s16x2_relu(a[i], k1, c[i]);
+        c[i] = __viaddmax_s16x2_relu(c[i], k2, a[i]);
+        asm volatile("add.s16x2 %0, %0, %1;" : "+r"(b[i]) : "r"(k1));
+        asm volatile("max.f16x2 %0, %0, %1;" : "+r"(b[i]) : "r"(a[i]));
       } else if constexpr (MIX == 7) {   // VIADDMNMX + SHFL-free SEL/LOP3
         a[i] = __viaddmax_s16x2_relu(a[i], k1, c[i]);
         asm volatile("lop3.b32 %0, %0, %1, %2, 0x96;" : "+r"(b[i]) : "r"(k2), "r"(c[i]));
@@ -89,5 +103,9 @@ int main() {
   run<5>("viaddmnmx+imad", 2, sms, d);
   run<6>("viaddmnmx+vimnmx+iadd", 3, sms, d);
   run<7>("viaddmnmx+lop3x2", 3, sms, d);
+  run<8>("hmnmx2+iadd", 2, sms, d);
+  run<9>("viaddmnmx+hmnmx2", 2, sms, d);
+  run<10>("viadd16x2+hmnmx2", 2, sms, d);
+  run<11>("2viaddmnmx+viadd16x2+hmnmx2", 4, sms, d);
   return 0;
 }

@@ -135,9 +135,9 @@ __device__ __forceinline__ void strip_pass(const uint8_t* sprof, int LS, int LB,
                                            uint2* __restrict__ wp, volatile int* prog_in, int need_base,
                                            volatile int* prog_out, int pub_base, uint32_t code_pad2, uint32_t nGe,
                                            uint32_t nGsGe, uint32_t& best, uint32_t shift = 0) {
-  uint32_t Hl[R], E[R];
+  uint32_t HA[R], HB[R], E[R];
 #pragma unroll
-  for (int r = 0; r < R; ++r) { Hl[r] = 0; E[r] = 0; }
+  for (int r = 0; r < R; ++r) { HA[r] = 0; HB[r] = 0; E[r] = 0; }
   uint32_t hdiag = 0, sH = 0, sF = 0, sC = code_pad2;
   const uint2* __restrict__ codes = reinterpret_cast<const uint2*>(pstream);
   const uint32_t pad4 = code_pad2 | (code_pad2 << 16);
@@ -188,14 +188,17 @@ __device__ __forceinline__ void strip_pass(const uint8_t* sprof, int LS, int LB,
         rH = tv.x;
         rF = tv.y;
       }
+      // even steps read HA and write HB, odd steps the reverse (4 steps per block)
       if constexpr (Q2) {
         // one DB sequence (byte `shift` of the pair word) against two queries
         const uint8_t* pa = sprof + ((rC >> shift) & 0xffu) * LS + laneoff;
-        gotoh_column_q2<R>(Hl, E, best, hdiag, pa, rH, rF, nGe, nGsGe);
+        if (j & 1) gotoh_column_q2<R>(HB, HA, E, best, hdiag, pa, rH, rF, nGe, nGsGe);
+        else gotoh_column_q2<R>(HA, HB, E, best, hdiag, pa, rH, rF, nGe, nGsGe);
       } else {
         const uint8_t* pa = sprof + (rC & 0xffu) * LS + laneoff;
         const uint8_t* pb = sprof + (rC >> 8) * LS + laneoff;
-        gotoh_column<R>(Hl, E, best, hdiag, pa, pb, rH, rF, nGe, nGsGe);
+        if (j & 1) gotoh_column<R>(HB, HA, E, best, hdiag, pa, pb, rH, rF, nGe, nGsGe);
+        else gotoh_column<R>(HA, HB, E, best, hdiag, pa, pb, rH, rF, nGe, nGsGe);
       }
       sH = rH;
       sF = rF;

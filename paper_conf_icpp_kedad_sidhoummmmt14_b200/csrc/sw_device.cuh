@@ -45,13 +45,15 @@ __host__ __device__ constexpr int lane_block_bytes(int R) {
 }
 
 // One column of R rows for one lane.
-//   Hl[r]  : in H_{r,j-1}, out H_{r,j}
+//   Hin[r] : H_{r,j-1} (previous column);  Hl[r] : out H_{r,j}  (caller alternates
+//            two buffers so the diagonal needs no register moves)
 //   E[r]   : in E_{r,j},   out E_{r,j+1}
 //   hdiag  : in H_{top-1, j-1}, out H_{top-1, j}  (top boundary of the previous column)
 //   Hio    : in H_{top-1, j} (from the lane above), out H_{bottom, j}
 //   Fio    : in F_{top, j},                        out F_{bottom+1, j}
 template <int R>
-__device__ __forceinline__ void gotoh_column(uint32_t (&Hl)[R], uint32_t (&E)[R], uint32_t& best,
+__device__ __forceinline__ void gotoh_column(const uint32_t (&Hin)[R], uint32_t (&Hl)[R], uint32_t (&E)[R],
+                                             uint32_t& best,
                                              uint32_t& hdiag, const uint8_t* __restrict__ pa,
                                              const uint8_t* __restrict__ pb, uint32_t& Hio, uint32_t& Fio,
                                              uint32_t nGe, uint32_t nGsGe) {
@@ -75,16 +77,20 @@ __device__ __forceinline__ void gotoh_column(uint32_t (&Hl)[R], uint32_t (&E)[R]
     for (int j = 0; j < UB; ++j) {
       const int r = u * UB + j;
       const uint32_t s = prmt(wa[j >> 2], wb[j >> 2], pair_sel(j & 3));
-      // Eq. (2): H = max(max(Hdiag + S, E), F); E, F >= 0 so the 0 term is implied.
-      // Folding E first keeps the row-to-row chain F -> H -> t -> F' at 3 ops.
-      const uint32_t h = __vmaxs2(__viaddmax_s16x2(hd, s, E[r]), F);
-      hd = Hl[r];
+      // Eq. (2): H = max(D, E, F) with D = Hdiag + S; E, F >= 0 so the 0 term is
+      // implied.  D goes to the FMA pipe (VIADD.16x2) and feeds both the 3-input
+      // max (VIMNMX3) and the running maximum: max over all D = max over all H
+      // (E and F never exceed an earlier H), so the ALU pipe carries only
+      // 1 + 1 + 1 + 1/2 = 3.5 ops per cell pair.
+      const uint32_t dg = __vadd2(hd, s);
+      const uint32_t h = __vimax3_s16x2(dg, E[r], F);
+      hd = Hin[r];  // ping-pong buffers: no register moves for the diagonal
       Hl[r] = h;
       const uint32_t t = __vadd2(h, nGsGe);                              // H - Gs - Ge
       E[r] = __viaddmax_s16x2_relu(E[r], nGe, t);                        // Eq. (3)
       F = __viaddmax_s16x2_relu(F, nGe, t);                              // Eq. (4)
-      if (r & 1) best = __vimax3_s16x2(best, hprev, h);
-      else hprev = h;
+      if (r & 1) best = __vimax3_s16x2(best, hprev, dg);
+      else hprev = dg;
     }
   }
   Hio = Hl[R - 1];
@@ -96,7 +102,8 @@ __device__ __forceinline__ void gotoh_column(uint32_t (&Hl)[R], uint32_t (&E)[R]
 // load, so no PRMT is needed: 5.5 DPX lane-ops per cell pair, of which the
 // VIADD.16x2 runs on the FMA pipe (4.5 on the ALU pipe).
 template <int R>
-__device__ __forceinline__ void gotoh_column_q2(uint32_t (&Hl)[R], uint32_t (&E)[R], uint32_t& best,
+__device__ __forceinline__ void gotoh_column_q2(const uint32_t (&Hin)[R], uint32_t (&Hl)[R], uint32_t (&E)[R],
+                                                uint32_t& best,
                                                 uint32_t& hdiag, const uint8_t* __restrict__ pa, uint32_t& Hio,
                                                 uint32_t& Fio, uint32_t nGe, uint32_t nGsGe) {
   static_assert(R % 4 == 0, "R must be a multiple of 4");
@@ -111,14 +118,15 @@ __device__ __forceinline__ void gotoh_column_q2(uint32_t (&Hl)[R], uint32_t (&E)
 #pragma unroll
     for (int j = 0; j < 4; ++j) {
       const int r = u * 4 + j;
-      const uint32_t h = __vmaxs2(__viaddmax_s16x2(hd, sv[j], E[r]), F);  // Eq. (2)
-      hd = Hl[r];
+      const uint32_t dg = __vadd2(hd, sv[j]);                              // FMA pipe
+      const uint32_t h = __vimax3_s16x2(dg, E[r], F);                       // Eq. (2)
+      hd = Hin[r];
       Hl[r] = h;
       const uint32_t t = __vadd2(h, nGsGe);
       E[r] = __viaddmax_s16x2_relu(E[r], nGe, t);                          // Eq. (3)
       F = __viaddmax_s16x2_relu(F, nGe, t);                                // Eq. (4)
-      if (r & 1) best = __vimax3_s16x2(best, hprev, h);
-      else hprev = h;
+      if (r & 1) best = __vimax3_s16x2(best, hprev, dg);                   // max D = max H
+      else hprev = dg;
     }
   }
   Hio = Hl[R - 1];

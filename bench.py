@@ -45,10 +45,12 @@ WORKLOADS = {
 REASONS = {0x1: "gpu_idle", 0x2: "applications_clocks_setting", 0x4: "sw_power_cap", 0x8: "hw_slowdown",
            0x10: "sync_boost", 0x20: "sw_thermal_slowdown", 0x40: "hw_thermal_slowdown",
            0x80: "hw_power_brake_slowdown", 0x100: "display_clock_setting"}
-# DPX ALU pipe: 64 lanes/clk/SM (16 per SMSP, measured by tools/dpx_microbench.cu: 18.4 T lane-ops/s);
-# the Gotoh s16x2 update needs 5.5 lane-ops per 2 cells.
+# The bound is the ALU pipe: 64 lanes/clk/SM (16 per SMSP; tools/dpx_microbench.cu measured 18.4 T
+# lane-ops/s for VIADDMNMX/VIMNMX3/PRMT on 148 SMs).  tools/pipe_mix.cu showed VIADD.16x2 issues on the
+# FMA pipe, so the minimal s16x2 Gotoh update puts 3.5 ALU-pipe ops on 2 cells: VIMNMX3 (H), 2x
+# VIADDMNMX.RELU (E', F'), 1/2 VIMNMX3 (running max) -> 1.75 per cell.
 ALU_LANES_PER_SM_CLK = 64
-OPS_PER_CELL = 2.75
+OPS_PER_CELL = 1.75
 
 
 def parse():
@@ -354,8 +356,9 @@ def run_ours(args):
                              "peak": round(peak, 1), "unit": "GCUPS", "frac": round(achieved / peak, 4) if achieved else None,
                              "traffic": traffic,
                              "kernel": "inter_kernel (short pairs), CUDA events around each launch",
-                             "peak_basis": f"{n_sm} SMs x {ALU_LANES_PER_SM_CLK} DPX lanes/clk x {sm_max:.0f} MHz / "
-                                           f"{OPS_PER_CELL} lane-ops per cell"},
+                             "peak_basis": f"{n_sm} SMs x {ALU_LANES_PER_SM_CLK} ALU-pipe lanes/clk x {sm_max:.0f} MHz / "
+                                           f"{OPS_PER_CELL} ALU lane-ops per cell (minimal s16x2 Gotoh update; "
+                                           f"derived from unit counts + measured pipe attribution)"},
                 "cpu_baseline": cpu, "e2e": e2e, "gpu_launches": int(n_launch_step * args.steps),
                 "clocks": clk,
                 "detail": {"search_ms_per_step": round(T / args.steps, 3),

@@ -64,6 +64,10 @@ def parse():
     ap.add_argument("--e2e-steps", type=int, default=2)
     ap.add_argument("--no-cpu-baseline", action="store_true")
     ap.add_argument("--cpu-baseline-cells", type=float, default=3.0e10)
+    ap.add_argument("--verify", type=int, default=0, help="after timing, check N sampled DB sequences "
+                    "of the assembled scores against the CPU oracle (rank 0)")
+    ap.add_argument("--dist-backend", default="nccl", help="nccl (default); gloo only for functional checks "
+                    "of the multi-rank path on a box with fewer GPUs than ranks")
     return ap.parse_args()
 
 
@@ -217,12 +221,17 @@ def run_ours(args):
     if world != args.gpus:
         if world == 1 and args.gpus > 1:
             raise SystemExit("--gpus N > 1 needs torchrun --nproc-per-node N")
+    if args.dist_backend == "gloo":
+        local = local % torch.cuda.device_count()  # functional check: ranks may share a GPU
     torch.cuda.set_device(local)
     dev = torch.device("cuda", local)
     pg = None
     if world > 1:
         import torch.distributed as tdist
-        tdist.init_process_group("nccl", device_id=dev)
+        if args.dist_backend == "nccl":
+            tdist.init_process_group("nccl", device_id=dev)
+        else:
+            tdist.init_process_group("gloo")
         pg = tdist
 
     def barrier():
@@ -258,11 +267,19 @@ def run_ours(args):
         jobs.append((s, qs, qc, qo, view))
     stream = torch.cuda.current_stream(dev)
 
+    def gather():
+        if args.dist_backend == "nccl":
+            pg.all_gather_into_tensor(gathered, flat)
+        else:  # gloo: host staging (functional checks only)
+            g = torch.empty(world * cap, dtype=torch.int32)
+            pg.all_gather_into_tensor(g, flat.cpu())
+            gathered.copy_(g)
+
     def step():
         for s, qs, qc, qo, view in jobs:
             h.search(qc, qo, dbs[s], S, 10, 2, out=view, stream=stream)
         if world > 1:
-            pg.all_gather_into_tensor(gathered, flat)
+            gather()
 
     for _ in range(args.warmup):
         step()
@@ -332,7 +349,7 @@ def run_ours(args):
             else:
                 for s, qs, qc, qo, view in jobs:
                     h.search(qc, qo, dbs[s], S, 10, 2, out=view, stream=stream)      # H2D of queries inside
-                pg.all_gather_into_tensor(gathered, flat)
+                gather()
                 if rank == 0:
                     final_host.copy_(gathered, non_blocking=False)
         torch.cuda.synchronize()
@@ -342,6 +359,24 @@ def run_ours(args):
             pg.all_reduce(dtt, op=pg.ReduceOp.MAX)
         e2e = {"value": round(total_cells * args.e2e_steps / float(dtt.item()) / 1e9, 2), "unit": "GCUPS",
                "h2d_bytes_per_step": h2d * world, "d2h_bytes_per_step": d2h}
+
+    verified = None
+    if args.verify > 0:
+        if world > 1:
+            gather()
+            torch.cuda.synchronize()
+        if rank == 0:
+            g = (gathered if world > 1 else flat).cpu().numpy().reshape(world, -1)
+            full = swdist.assemble(plan, Q, N, [g[r] for r in range(world)])
+            import oracle
+            from oracle.blosum62 import blosum62 as ob62
+            rng = np.random.default_rng(5)
+            idx = np.sort(rng.choice(N, size=min(N, args.verify), replace=False))
+            sc, so = swdist.subset(c["dcodes"], c["doff"], idx)
+            ref = oracle.gotoh_search(c["qcodes"], c["qoff"], sc, so, ob62(), 10, 2, procs=os.cpu_count() or 1)
+            verified = bool(np.array_equal(full[:, idx], ref))
+            if not verified:
+                raise SystemExit(f"verify: {int((full[:, idx] != ref).sum())} mismatches vs oracle")
 
     cpu = None
     if rank == 0 and world == 1 and not args.no_cpu_baseline:
@@ -360,6 +395,7 @@ def run_ours(args):
                                            f"{OPS_PER_CELL} ALU lane-ops per cell (minimal s16x2 Gotoh update; "
                                            f"derived from unit counts + measured pipe attribution)"},
                 "cpu_baseline": cpu, "e2e": e2e, "gpu_launches": int(n_launch_step * args.steps),
+                **({"verified_sample": args.verify, "verified": verified} if args.verify else {}),
                 "clocks": clk,
                 "detail": {"search_ms_per_step": round(T / args.steps, 3),
                            "short_kernel_ms_per_step": round(st["short_ms"] / args.steps, 3),

@@ -344,7 +344,7 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
   int G = 4, R = 24;
   choose_geom(h, slot_m, nshort > 0 ? c.sum_short / nshort : 1.0, G, R);
   if (!inter_config_supported(G, R)) fail(SW_EUNSUPPORTED, "no kernel for this geometry");
-  const int NT = 256, NG = NT / G, W = NT / 32;
+  const int NT = inter_block_threads(), NG = NT / G, W = NT / 32;
   const int LB2 = (((R / 4) | 1) * 16);
   const int LS2 = G * LB2;
   const int SB2 = (((alpha + 1) * LS2 + 15) / 16) * 16;
@@ -439,9 +439,9 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
   for (auto& x : gs) max_strips = std::max(max_strips, x.n_strips);
   int max_lstrips = 1;
   for (auto& x : gl) max_lstrips = std::max(max_lstrips, x.n_strips);
-  const int bcap = c.max_short + G + 8;
+  const int bcap = c.max_short + 2 * G + 8;  // wave width up to 2G sub-lanes
   if (max_strips > 1 && nshort > 0) SW_CK(h->bbuf.ensure(size_t(grid) * NG * bcap * sizeof(uint2)));
-  const int lcap = c.max_long + 32 + 8;
+  const int lcap = c.max_long + 64 + 8;
   if (nlong > 0 && max_lstrips > 1) SW_CK(h->bbuf_long.ensure(size_t(grid) * W * lcap * sizeof(uint2)));
   SW_CK(h->counters.ensure(sizeof(int)));
   SW_CK(cudaMemsetAsync(h->counters.p, 0, sizeof(int), c.st));

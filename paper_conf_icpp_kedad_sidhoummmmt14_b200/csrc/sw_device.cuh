@@ -44,92 +44,65 @@ __host__ __device__ constexpr int lane_block_bytes(int R) {
   return ((R % 8 == 0) ? (((R / 8) | 1) * 8) : (((R / 4) | 1) * 4));
 }
 
-// One column of R rows for one lane.
-//   Hin[r] : H_{r,j-1} (previous column);  Hl[r] : out H_{r,j}  (caller alternates
-//            two buffers so the diagonal needs no register moves)
+// Rows [R0, R1) of one column for one lane (a "sub-lane"; R0 = 0, R1 = R is
+// the whole lane).
+//   Hin[r] : H_{r,j-1} (previous column);  Hout[r] : out H_{r,j}  (the caller
+//            alternates two buffers, so the diagonal needs no register moves)
 //   E[r]   : in E_{r,j},   out E_{r,j+1}
-//   hdiag  : in H_{top-1, j-1}, out H_{top-1, j}  (top boundary of the previous column)
-//   Hio    : in H_{top-1, j} (from the lane above), out H_{bottom, j}
-//   Fio    : in F_{top, j},                        out F_{bottom+1, j}
-template <int R>
-__device__ __forceinline__ void gotoh_column(const uint32_t (&Hin)[R], uint32_t (&Hl)[R], uint32_t (&E)[R],
-                                             uint32_t& best,
-                                             uint32_t& hdiag, const uint8_t* __restrict__ pa,
-                                             const uint8_t* __restrict__ pb, uint32_t& Hio, uint32_t& Fio,
-                                             uint32_t nGe, uint32_t nGsGe) {
+//   hdiag  : in H_{R0-1, j-1}, out H_{R0-1, j}  (top boundary of the previous column)
+//   Hio    : in H_{R0-1, j} (from above), out H_{R1-1, j}
+//   Fio    : in F_{R0, j},                out F_{R1, j}
+// Q2 = false: pa / pb point at the int8 profile rows of the two DB letters of a
+//   pair (one per s16x2 half), combined per row by a sign-extending PRMT.
+// Q2 = true:  pa points at s16x2 profile words (two queries, one DB letter).
+template <int R, int R0, int R1, bool Q2>
+__device__ __forceinline__ void gotoh_rows(const uint32_t (&Hin)[R], uint32_t (&Hout)[R], uint32_t (&E)[R],
+                                           uint32_t& best, uint32_t& hdiag, const uint8_t* __restrict__ pa,
+                                           const uint8_t* __restrict__ pb, uint32_t& Hio, uint32_t& Fio,
+                                           uint32_t nGe, uint32_t nGsGe) {
+  static_assert(R0 % 4 == 0 && (R1 - R0) % 4 == 0 && R1 <= R, "row range must be 4-aligned");
   uint32_t hd = hdiag;
   hdiag = Hio;
   uint32_t F = Fio;
-  uint32_t hprev = 0;
-  constexpr int UB = ProfUnit<R>::BYTES;
+  uint32_t dprev = 0;
+  constexpr int UB = Q2 ? 4 : ((R % 8 == 0 && R0 % 8 == 0 && (R1 - R0) % 8 == 0) ? 8 : 4);  // rows per load
 #pragma unroll
-  for (int u = 0; u < R / UB; ++u) {
-    uint32_t wa[UB / 4], wb[UB / 4];
-    if constexpr (UB == 8) {
+  for (int u = R0 / UB; u < R1 / UB; ++u) {
+    uint32_t sv[UB];
+    if constexpr (Q2) {
+      const uint4 w = *reinterpret_cast<const uint4*>(pa + u * 16);
+      sv[0] = w.x; sv[1] = w.y; sv[2] = w.z; sv[3] = w.w;
+    } else if constexpr (UB == 8) {
       const uint2 x = *reinterpret_cast<const uint2*>(pa + u * 8);
       const uint2 y = *reinterpret_cast<const uint2*>(pb + u * 8);
-      wa[0] = x.x; wa[1] = x.y; wb[0] = y.x; wb[1] = y.y;
+#pragma unroll
+      for (int j = 0; j < 8; ++j) sv[j] = prmt(j < 4 ? x.x : x.y, j < 4 ? y.x : y.y, pair_sel(j & 3));
     } else {
-      wa[0] = *reinterpret_cast<const uint32_t*>(pa + u * 4);
-      wb[0] = *reinterpret_cast<const uint32_t*>(pb + u * 4);
+      const uint32_t x = *reinterpret_cast<const uint32_t*>(pa + u * 4);
+      const uint32_t y = *reinterpret_cast<const uint32_t*>(pb + u * 4);
+#pragma unroll
+      for (int j = 0; j < 4; ++j) sv[j] = prmt(x, y, pair_sel(j));
     }
 #pragma unroll
     for (int j = 0; j < UB; ++j) {
       const int r = u * UB + j;
-      const uint32_t s = prmt(wa[j >> 2], wb[j >> 2], pair_sel(j & 3));
       // Eq. (2): H = max(D, E, F) with D = Hdiag + S; E, F >= 0 so the 0 term is
       // implied.  D goes to the FMA pipe (VIADD.16x2) and feeds both the 3-input
       // max (VIMNMX3) and the running maximum: max over all D = max over all H
       // (E and F never exceed an earlier H), so the ALU pipe carries only
       // 1 + 1 + 1 + 1/2 = 3.5 ops per cell pair.
-      const uint32_t dg = __vadd2(hd, s);
+      const uint32_t dg = __vadd2(hd, sv[j]);
       const uint32_t h = __vimax3_s16x2(dg, E[r], F);
-      hd = Hin[r];  // ping-pong buffers: no register moves for the diagonal
-      Hl[r] = h;
+      hd = Hin[r];
+      Hout[r] = h;
       const uint32_t t = __vadd2(h, nGsGe);                              // H - Gs - Ge
       E[r] = __viaddmax_s16x2_relu(E[r], nGe, t);                        // Eq. (3)
       F = __viaddmax_s16x2_relu(F, nGe, t);                              // Eq. (4)
-      if (r & 1) best = __vimax3_s16x2(best, hprev, dg);
-      else hprev = dg;
+      if (r & 1) best = __vimax3_s16x2(best, dprev, dg);
+      else dprev = dg;
     }
   }
-  Hio = Hl[R - 1];
-  Fio = F;
-}
-
-// Query-pair variant (two QUERIES per register, one DB sequence): the profile
-// already holds (S[qA_i][a], S[qB_i][a]) as s16x2 words, 4 rows per 16-byte
-// load, so no PRMT is needed: 5.5 DPX lane-ops per cell pair, of which the
-// VIADD.16x2 runs on the FMA pipe (4.5 on the ALU pipe).
-template <int R>
-__device__ __forceinline__ void gotoh_column_q2(const uint32_t (&Hin)[R], uint32_t (&Hl)[R], uint32_t (&E)[R],
-                                                uint32_t& best,
-                                                uint32_t& hdiag, const uint8_t* __restrict__ pa, uint32_t& Hio,
-                                                uint32_t& Fio, uint32_t nGe, uint32_t nGsGe) {
-  static_assert(R % 4 == 0, "R must be a multiple of 4");
-  uint32_t hd = hdiag;
-  hdiag = Hio;
-  uint32_t F = Fio;
-  uint32_t hprev = 0;
-#pragma unroll
-  for (int u = 0; u < R / 4; ++u) {
-    const uint4 w = *reinterpret_cast<const uint4*>(pa + u * 16);
-    const uint32_t sv[4] = {w.x, w.y, w.z, w.w};
-#pragma unroll
-    for (int j = 0; j < 4; ++j) {
-      const int r = u * 4 + j;
-      const uint32_t dg = __vadd2(hd, sv[j]);                              // FMA pipe
-      const uint32_t h = __vimax3_s16x2(dg, E[r], F);                       // Eq. (2)
-      hd = Hin[r];
-      Hl[r] = h;
-      const uint32_t t = __vadd2(h, nGsGe);
-      E[r] = __viaddmax_s16x2_relu(E[r], nGe, t);                          // Eq. (3)
-      F = __viaddmax_s16x2_relu(F, nGe, t);                                // Eq. (4)
-      if (r & 1) best = __vimax3_s16x2(best, hprev, dg);                   // max D = max H
-      else hprev = dg;
-    }
-  }
-  Hio = Hl[R - 1];
+  Hio = Hout[R1 - 1];
   Fio = F;
 }
 

@@ -125,6 +125,7 @@ cudaError_t launch_build_profile_q2(const uint8_t* qa, int ma, const uint8_t* qb
 int inter_max_ctas_per_sm(int G, int R, int NT, int smem_bytes);
 cudaError_t launch_inter(int G, int R, int NT, int grid, int smem_bytes, const InterArgs& a, cudaStream_t st);
 bool inter_config_supported(int G, int R);
+int inter_block_threads();  // NT of the scoring kernel (its long items use NT/32 chained warps)
 cudaError_t launch_rescore(int grid, const RescoreArgs& a, cudaStream_t st);
 constexpr int RESCORE_WARPS = 16;
 constexpr int RESCORE_R = 8;

@@ -301,7 +301,8 @@ def run_ours(args):
     clk = clocks.stop()
     ms_local = e0.elapsed_time(e1)
     st = h.last_stats()
-    ms = torch.tensor([ms_local], dtype=torch.float64, device=dev)
+    cdev = dev if args.dist_backend == "nccl" else torch.device("cpu")
+    ms = torch.tensor([ms_local], dtype=torch.float64, device=cdev)
     if pg is not None:
         pg.all_reduce(ms, op=pg.ReduceOp.MAX)
     T = float(ms.item())
@@ -318,6 +319,10 @@ def run_ours(args):
         cells_short_step += one["cells_short"]
         n_launch_step += one["n_launches"]
     torch.cuda.synchronize()
+    if pg is not None:  # launches of every rank (the whole job)
+        nl = torch.tensor([n_launch_step], dtype=torch.int64, device=cdev)
+        pg.all_reduce(nl)
+        n_launch_step = int(nl.item())
     sm_max = clk.get("sm_max_mhz") or 1965.0
     n_sm = torch.cuda.get_device_properties(dev).multi_processor_count
     peak = n_sm * ALU_LANES_PER_SM_CLK * sm_max * 1e6 / OPS_PER_CELL / 1e9
@@ -354,7 +359,7 @@ def run_ours(args):
                     final_host.copy_(gathered, non_blocking=False)
         torch.cuda.synchronize()
         dt = time.perf_counter() - t0
-        dtt = torch.tensor([dt], dtype=torch.float64, device=dev)
+        dtt = torch.tensor([dt], dtype=torch.float64, device=cdev)
         if pg is not None:
             pg.all_reduce(dtt, op=pg.ReduceOp.MAX)
         e2e = {"value": round(total_cells * args.e2e_steps / float(dtt.item()) / 1e9, 2), "unit": "GCUPS",

@@ -109,6 +109,9 @@ struct sw_db_s {
   std::vector<int64_t> seq_len;  // caller order
   std::vector<int64_t> sorted_lens;  // descending, non-empty only (for overflow bounds)
   int n_long = 0;                // pairs [0, n_long) have len > T_LONG
+  // per-DB constants of the pair table (computed once at load)
+  double sum_short_len = 0, sum_long_len = 0, short_res = 0;
+  int32_t max_short = 0, max_long = 0;
   DevBuf stream, dpairs;
 };
 
@@ -135,11 +138,11 @@ static int32_t guarded(sw_handle_s* h, F&& f) {
 // ----------------------------------------------------------------------------
 // geometry of the inter-task kernel for a query of m rows and a launch whose
 // pairs average Lavg columns
-static ProfGeom make_geom(int G, int R, int m, int alpha) {
+static ProfGeom make_geom(int G, int R, int m, int alpha, bool dense = false) {
   ProfGeom g{};
   g.G = G;
   g.R = R;
-  g.LB = ((R % 8 == 0) ? (((R / 8) | 1) * 8) : (((R / 4) | 1) * 4));
+  g.LB = dense ? R : ((R % 8 == 0) ? (((R / 8) | 1) * 8) : (((R / 4) | 1) * 4));
   g.LS = G * g.LB;
   g.NL = alpha + 1;
   g.SB = ((g.NL * g.LS + 15) / 16) * 16;
@@ -259,6 +262,17 @@ int32_t sw_load_db(sw_handle_t h, const uint8_t* codes, const int64_t* offsets, 
     db->seq_len = std::move(P.seq_len);
     db->sorted_lens = std::move(P.sorted_lens);
     const size_t np = db->pairs.size();
+    for (size_t p = 0; p < np; ++p) {
+      const PairRec& r = db->pairs[p];
+      if (int(p) < db->n_long) {
+        db->sum_long_len += r.len;
+        db->max_long = std::max(db->max_long, r.len);
+      } else {
+        db->sum_short_len += r.len;
+        db->max_short = std::max(db->max_short, r.len);
+        db->short_res += double(db->seq_len[size_t(r.id0)]) + (r.id1 >= 0 ? double(db->seq_len[size_t(r.id1)]) : 0.0);
+      }
+    }
     std::vector<uint16_t>& stream = P.stream;
     SW_CK(db->stream.ensure(stream.size() * sizeof(uint16_t)));
     SW_CK(db->dpairs.ensure(std::max<size_t>(np, 1) * sizeof(PairRec)));
@@ -353,7 +367,7 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
   std::vector<ProfGeom> gl;
   std::vector<size_t> off_l;
   for (int m : ms) {
-    gl.push_back(make_geom(32, LONG_R, m, alpha));
+    gl.push_back(make_geom(32, LONG_R, m, alpha, /*dense=*/true));
     off_l.push_back(total);
     total += nlong > 0 ? size_t(gl.back().n_strips) * gl.back().SB : 0;
   }
@@ -371,11 +385,7 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
   const int8_t* dmat = h->matrix.as<int8_t>();
   auto qptr = [&](int k) { return h->qcodes.as<uint8_t>() + qoff0[size_t(order[size_t(k)])]; };
   std::vector<QueryDesc> desc(order.size());
-  double sumS = 0, sumL = 0;
-  for (int p = 0; p < np; ++p) {
-    if (p < nlong) sumL += db->pairs[size_t(p)].len + 32;
-    else sumS += db->pairs[size_t(p)].len + G;
-  }
+  const double sumS = db->sum_short_len + double(nshort) * G, sumL = db->sum_long_len + double(nlong) * 32;
   for (size_t k = 0; k < order.size(); ++k) {
     const int qi = order[k];
     if (nlong > 0) {
@@ -572,15 +582,8 @@ int32_t sw_search(sw_handle_t h, const uint8_t* q_codes, const int64_t* q_offset
     SW_CK(h->ovf.ensure(size_t(std::max<int64_t>(ovf_cap, 1)) * sizeof(OvfRec)));
     SW_CK(h->ovf_count.ensure(sizeof(int)));
     SW_CK(cudaMemsetAsync(h->ovf_count.p, 0, sizeof(int), st));
-    const int np = int(db->pairs.size());
-    const int nlong = db->n_long;
-    double sum_short = 0;
-    int32_t max_short = 0, max_long = 0;
-    for (int p = 0; p < np; ++p) {
-      const int32_t L = db->pairs[size_t(p)].len;
-      if (p < nlong) max_long = std::max(max_long, L);
-      else { sum_short += L; max_short = std::max(max_short, L); }
-    }
+    const double sum_short = db->sum_short_len;
+    const int32_t max_short = db->max_short, max_long = db->max_long;
     const uint32_t nGe16 = uint32_t(uint16_t(int16_t(-gap_extend)));
     const uint32_t nGsGe16 = uint32_t(uint16_t(int16_t(-(gap_open + gap_extend))));
     LaunchCtx lc{};
@@ -635,11 +638,7 @@ int32_t sw_search(sw_handle_t h, const uint8_t* q_codes, const int64_t* q_offset
     double sq = 0;
     for (auto L : qlen) sq += double(L);
     h->stats.cells = sq * double(db->n_res);
-    double short_res = 0;
-    for (int p = nlong; p < np; ++p) {
-      const PairRec& r = db->pairs[size_t(p)];
-      short_res += double(db->seq_len[size_t(r.id0)]) + (r.id1 >= 0 ? double(db->seq_len[size_t(r.id1)]) : 0.0);
-    }
+    const double short_res = db->short_res;
     h->stats.cells_short = sq * short_res;  // pairs <= 3000 columns (inter-task mode)
     h->stats.cells_computed = cells_computed;
     h->stats.n_launches = launches;

@@ -107,13 +107,24 @@ cudaError_t launch_build_profile_q2(const uint8_t* qa, int ma, const uint8_t* qb
 // Warp-uniform wait until a shared progress counter reaches `need` (all lanes
 // read the broadcast word; __all_sync keeps the warp converged so the shuffles
 // that follow stay on the fast path), then a CTA-scope acquire fence.
+__device__ __forceinline__ int ld_acquire_cta(const volatile int* p) {
+  int v;
+  asm volatile("ld.acquire.cta.shared.b32 %0, [%1];"
+               : "=r"(v) : "r"(static_cast<uint32_t>(__cvta_generic_to_shared(const_cast<int*>(p)))) : "memory");
+  return v;
+}
+
+__device__ __forceinline__ void st_release_cta(volatile int* p, int v) {
+  asm volatile("st.release.cta.shared.b32 [%0], %1;"
+               :: "r"(static_cast<uint32_t>(__cvta_generic_to_shared(const_cast<int*>(p)))), "r"(v) : "memory");
+}
+
 __device__ __forceinline__ void wait_progress(volatile int* p, int need) {
   for (;;) {
-    const int v = *p;
+    const int v = ld_acquire_cta(p);  // acquire: later link reads see the producer's writes
     if (__all_sync(FULL, v >= need)) break;
     __nanosleep(100);
   }
-  __threadfence_block();
 }
 
 // ---------------------------------------------------------------------------
@@ -244,13 +255,7 @@ __device__ __forceinline__ void strip_pass(const uint8_t* sprof, int LS, int LB,
       }
     }
     wp += 4;
-    if (LINKED && wr) {
-      __syncwarp();
-      if (tail) {
-        __threadfence_block();
-        *prog_out = pub_base + t0 + 4;
-      }
-    }
+    if (LINKED && wr && tail) st_release_cta(prog_out, pub_base + t0 + 4);  // orders this lane's link writes
   }
 }
 
@@ -573,10 +578,7 @@ __global__ void __launch_bounds__(RESCORE_WARPS * 32) rescore_kernel(RescoreArgs
           sC = rC;
           if (wr && tail) __stcg(wp + t0 + j, make_int2(sH, sF));
         }
-        if (wr) {
-          __syncwarp();
-          if (tail) { __threadfence_block(); *pout = pub_base + t0 + 4; }
-        }
+        if (wr && tail) st_release_cta(pout, pub_base + t0 + 4);
       }
     }
 #pragma unroll

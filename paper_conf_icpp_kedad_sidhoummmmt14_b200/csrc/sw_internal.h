@@ -48,7 +48,8 @@ struct ProfGeom {
   int n_strips;    // ceil(m / (G*R))
 };
 
-constexpr int LONG_R = 8;    // rows per lane of the intra-task (long pair) geometry, G = 32
+constexpr int LONG_R = 16;   // rows per lane of the intra-task (long pair) geometry, G = 32;
+                             // lane block = LONG_R bytes (no bank padding: 8 strip slots must fit in smem)
 
 // Per-query descriptor of a multi-query launch (processing order: longest first).
 struct QueryDesc {

@@ -71,7 +71,8 @@ struct SwError {
 
 [[noreturn]] void fail(int32_t code, const std::string& m) { throw SwError{code, m}; }
 
-constexpr int T_LONG = 3000;  // pairs longer than this are launched separately
+constexpr int T_LONG = 3000;
+constexpr int LONG_ROUNDS = 3;  // target rounds of W strips per CTA for a long pair  // pairs longer than this are launched separately
 
 }  // namespace
 
@@ -85,6 +86,7 @@ struct sw_handle_s {
   std::vector<sw_db_s*> dbs;
   // scratch (grown on demand)
   DevBuf qcodes, qoff, matrix, prof, bbuf, bbuf_long, counters, ovf, ovf_count, scores_tmp, rbuf, qdesc;
+  DevBuf glinks, gflags;  // superstrip boundary rows and their counters (long pairs)
   cudaEvent_t ev_begin = nullptr, ev_end = nullptr;
   bool search_timed = false;
   bool timing_accumulate = false;
@@ -112,6 +114,8 @@ struct sw_db_s {
   // per-DB constants of the pair table (computed once at load)
   double sum_short_len = 0, sum_long_len = 0, short_res = 0;
   int32_t max_short = 0, max_long = 0;
+  int64_t glink_stride = 0;      // sum over long pairs of (len + 72): one superstrip boundary row set
+  DevBuf dlofs;                  // per long pair: offset of its boundary row
   DevBuf stream, dpairs;
 };
 
@@ -274,6 +278,14 @@ int32_t sw_load_db(sw_handle_t h, const uint8_t* codes, const int64_t* offsets, 
       }
     }
     std::vector<uint16_t>& stream = P.stream;
+    {
+      std::vector<int64_t> lofs(size_t(std::max(db->n_long, 1)), 0);
+      int64_t acc = 0;
+      for (int p = 0; p < db->n_long; ++p) { lofs[size_t(p)] = acc; acc += db->pairs[size_t(p)].len + 72; }
+      db->glink_stride = acc;
+      SW_CK(db->dlofs.ensure(lofs.size() * sizeof(int64_t)));
+      SW_CK(cudaMemcpyAsync(db->dlofs.p, lofs.data(), lofs.size() * sizeof(int64_t), cudaMemcpyHostToDevice, st));
+    }
     SW_CK(db->stream.ensure(stream.size() * sizeof(uint16_t)));
     SW_CK(db->dpairs.ensure(std::max<size_t>(np, 1) * sizeof(PairRec)));
     SW_CK(cudaMemcpyAsync(db->stream.p, stream.data(), stream.size() * sizeof(uint16_t), cudaMemcpyHostToDevice, st));
@@ -385,6 +397,7 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
   const int8_t* dmat = h->matrix.as<int8_t>();
   auto qptr = [&](int k) { return h->qcodes.as<uint8_t>() + qoff0[size_t(order[size_t(k)])]; };
   std::vector<QueryDesc> desc(order.size());
+  int64_t long_items = 0, flags_total = 0, glink_total = 0;
   const double sumS = db->sum_short_len + double(nshort) * G, sumL = db->sum_long_len + double(nlong) * 32;
   for (size_t k = 0; k < order.size(); ++k) {
     const int qi = order[k];
@@ -399,7 +412,17 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
     d.n_strips = 0;
     d.n_strips_long = gl[k].n_strips;
     d.qidx = qi;
+    // CTAs per long pair: enough to split very tall queries, few enough that each
+    // CTA still runs ~LONG_ROUNDS rounds of W strips (amortises the pipeline ramp)
+    d.n_super = std::max(1, (gl[k].n_strips + W * LONG_ROUNDS - 1) / (W * LONG_ROUNDS));
+    d.long_item_begin = int(long_items);
+    d.flag_base = int(flags_total);
+    d.done_base = int(k) * nlong;
     d.pad_ = 0;
+    d.glink_base = glink_total;
+    long_items += int64_t(nlong) * d.n_super;
+    flags_total += int64_t(nlong) * d.n_super;
+    if (d.n_super > 1) glink_total += int64_t(d.n_super) * db->glink_stride;
     cells_computed += 2.0 * sumL * double(gl[k].n_strips) * 32 * LONG_R;
   }
   std::vector<SlotDesc> sdesc(slots.size());
@@ -442,7 +465,7 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
   const int smem = std::max(g0.SB, SB2) + (nlong > 0 ? W * l0.SB : 0);
   const int occ = inter_max_ctas_per_sm(G, R, NT, smem);
   if (occ <= 0) fail(SW_ECUDA, "inter kernel does not fit on an SM");
-  const int64_t n_items = int64_t(order.size()) * nlong + item;
+  const int64_t n_items = long_items + item;
   if (n_items >= (int64_t(1) << 31)) fail(SW_EUNSUPPORTED, "too many work items");
   const int grid = int(std::max<int64_t>(1, std::min<int64_t>(n_items, int64_t(occ) * h->sms)));
   int max_strips = 1;
@@ -455,6 +478,10 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
   if (nlong > 0 && max_lstrips > 1) SW_CK(h->bbuf_long.ensure(size_t(grid) * W * lcap * sizeof(uint2)));
   SW_CK(h->counters.ensure(sizeof(int)));
   SW_CK(cudaMemsetAsync(h->counters.p, 0, sizeof(int), c.st));
+  const size_t nflags = size_t(std::max<int64_t>(flags_total, 1)), ndone = size_t(std::max<int64_t>(int64_t(order.size()) * nlong, 1));
+  SW_CK(h->gflags.ensure((nflags + ndone) * sizeof(int)));
+  SW_CK(cudaMemsetAsync(h->gflags.p, 0, (nflags + ndone) * sizeof(int), c.st));
+  if (glink_total > 0) SW_CK(h->glinks.ensure(size_t(glink_total) * sizeof(uint2)));
   InterArgs a{};
   a.queries = d_desc;
   a.n_queries = int(order.size());
@@ -471,6 +498,12 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
   a.LSL = l0.LS;
   a.LBL = l0.LB;
   a.n_long = nlong;
+  a.n_long_items = int(long_items);
+  a.glinks = glink_total > 0 ? h->glinks.as<uint2>() : nullptr;
+  a.gflags = h->gflags.as<int>();
+  a.gdone = h->gflags.as<int>() + nflags;
+  a.lofs = db->dlofs.as<int64_t>();
+  a.glink_stride = db->glink_stride;
   a.links = (nlong > 0 && max_lstrips > 1) ? h->bbuf_long.as<uint2>() : nullptr;
   a.lcap = lcap;
   a.stream = db->stream.as<uint16_t>();

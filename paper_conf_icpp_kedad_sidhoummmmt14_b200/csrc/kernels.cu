@@ -104,27 +104,52 @@ cudaError_t launch_build_profile_q2(const uint8_t* qa, int ma, const uint8_t* qb
   return cudaGetLastError();
 }
 
-// Warp-uniform wait until a shared progress counter reaches `need` (all lanes
-// read the broadcast word; __all_sync keeps the warp converged so the shuffles
-// that follow stay on the fast path), then a CTA-scope acquire fence.
-__device__ __forceinline__ int ld_acquire_cta(const volatile int* p) {
+// Progress counters of chained strips.  Within a CTA they live in shared memory
+// (CTA-scope release/acquire); between the CTAs that hold consecutive
+// "superstrips" of one long pair they live in global memory (GPU scope).
+__device__ __forceinline__ int ld_acquire_cta(const int* p) {
   int v;
   asm volatile("ld.acquire.cta.shared.b32 %0, [%1];"
                : "=r"(v) : "r"(static_cast<uint32_t>(__cvta_generic_to_shared(const_cast<int*>(p)))) : "memory");
   return v;
 }
-
-__device__ __forceinline__ void st_release_cta(volatile int* p, int v) {
+__device__ __forceinline__ void st_release_cta(int* p, int v) {
   asm volatile("st.release.cta.shared.b32 [%0], %1;"
-               :: "r"(static_cast<uint32_t>(__cvta_generic_to_shared(const_cast<int*>(p)))), "r"(v) : "memory");
+               :: "r"(static_cast<uint32_t>(__cvta_generic_to_shared(p))), "r"(v) : "memory");
+}
+__device__ __forceinline__ int ld_acquire_gpu(const int* p) {
+  int v;
+  asm volatile("ld.acquire.gpu.global.b32 %0, [%1];" : "=r"(v) : "l"(p) : "memory");
+  return v;
+}
+__device__ __forceinline__ void st_release_gpu(int* p, int v) {
+  asm volatile("st.release.gpu.global.b32 [%0], %1;" :: "l"(p), "r"(v) : "memory");
 }
 
-__device__ __forceinline__ void wait_progress(volatile int* p, int need) {
+// Link of a chained strip: the row above (read by lane 0) and this strip's
+// bottom row (written by the last lane), each with a progress counter.
+struct Link {
+  int* in;        // counter of the producer of the row above (nullptr: none)
+  int in_base;    // value the producer publishes before its first cell
+  bool in_gpu;    // counter in global memory (other CTA)
+  int* out;       // this strip's counter (nullptr: nobody consumes it)
+  int out_base;
+  bool out_gpu;
+};
+
+// Warp-uniform wait until a progress counter reaches `need` (one lane polls,
+// the result is broadcast, so the warp stays converged and the shuffles that
+// follow stay on the fast path).  `seen` caches the last value observed.
+__device__ __forceinline__ void wait_progress(const Link& lk, int need, int& seen) {
+  if (seen >= need) return;
   for (;;) {
-    const int v = ld_acquire_cta(p);  // acquire: later link reads see the producer's writes
-    if (__all_sync(FULL, v >= need)) break;
-    __nanosleep(100);
+    int v = 0;
+    if ((threadIdx.x & 31) == 0) v = lk.in_gpu ? ld_acquire_gpu(lk.in) : ld_acquire_cta(lk.in);
+    v = __shfl_sync(FULL, v, 0);
+    if (v >= need) { seen = v; break; }
+    __nanosleep(lk.in_gpu ? 256 : 64);
   }
+  if (lk.in_gpu) __threadfence();  // lane 0 acquired; make the row visible to its later loads
 }
 
 // ---------------------------------------------------------------------------
@@ -151,9 +176,8 @@ struct SubLanes {
 template <int G, int R, bool LINKED, bool Q2 = false>
 __device__ __forceinline__ void strip_pass(const uint8_t* sprof, int LS, int LB, const uint16_t* pstream, int L,
                                            int T, int k, bool rd, bool wr, const uint2* __restrict__ rp,
-                                           uint2* __restrict__ wp, volatile int* prog_in, int need_base,
-                                           volatile int* prog_out, int pub_base, uint32_t code_pad2, uint32_t nGe,
-                                           uint32_t nGsGe, uint32_t& best, uint32_t shift = 0) {
+                                           uint2* __restrict__ wp, const Link& lk, uint32_t code_pad2,
+                                           uint32_t nGe, uint32_t nGsGe, uint32_t& best, uint32_t shift = 0) {
   constexpr int V = SubLanes<R>::V;
   constexpr int VG = V * G;   // width of the wave in sub-lanes
   constexpr int RH = R / V;   // rows per sub-lane
@@ -176,7 +200,8 @@ __device__ __forceinline__ void strip_pass(const uint8_t* sprof, int LS, int LB,
   // L and t0 are multiples of 4, so one compare guards a whole block.
   uint2 cw = make_uint2(pad4, pad4);
   uint2 tb0 = z2, tb1 = z2, tb2 = z2, tb3 = z2;
-  if (LINKED && rd && L > 0) wait_progress(prog_in, need_base + min(4 + VG - 1 + LINK_LAG, L + VG));
+  int seen = -1;
+  if (LINKED && rd && L > 0) wait_progress(lk, lk.in_base + min(4 + VG - 1 + LINK_LAG, L + VG), seen);
   if (lead && L > 0) {
     cw = codes[0];
     if (rd) {
@@ -189,7 +214,7 @@ __device__ __forceinline__ void strip_pass(const uint8_t* sprof, int LS, int LB,
     const uint2 cwc = cw;
     const uint2 c0 = tb0, c1 = tb1, c2 = tb2, c3 = tb3;
     rp += 4;
-    if (LINKED && rd && t0 + 4 < L) wait_progress(prog_in, need_base + min(t0 + 8 + VG - 1 + LINK_LAG, L + VG));
+    if (LINKED && rd && t0 + 4 < L) wait_progress(lk, lk.in_base + min(t0 + 8 + VG - 1 + LINK_LAG, L + VG), seen);
     if (lead) {
       if (t0 + 4 < L) {
         cw = codes[(t0 + 4) >> 2];
@@ -255,7 +280,10 @@ __device__ __forceinline__ void strip_pass(const uint8_t* sprof, int LS, int LB,
       }
     }
     wp += 4;
-    if (LINKED && wr && tail) st_release_cta(prog_out, pub_base + t0 + 4);  // orders this lane's link writes
+    if (LINKED && wr && tail) {  // release orders this lane's link writes before the counter
+      if (!lk.out_gpu) st_release_cta(lk.out, lk.out_base + t0 + 4);
+      else if (((t0 >> 2) & 3) == 3 || t0 + 4 >= T) st_release_gpu(lk.out, lk.out_base + t0 + 4);
+    }
   }
 }
 
@@ -300,7 +328,7 @@ __global__ void __launch_bounds__(NT) inter_kernel(InterArgs a) {
   const int k = tid & (G - 1);
   const int g = tid / G;
   const int lane = tid & 31, warp = tid >> 5;
-  const int n_long_items = a.n_queries * a.n_long;
+  const int n_long_items = a.n_long_items;
   const int n_items = n_long_items + a.n_short_items;
   uint2* __restrict__ bb = a.bbuf + ((size_t)blockIdx.x * NG + g) * (size_t)a.bcap;
   int loaded = -1;  // (query rank << 16 | strip) of the short profile in shared memory (CTA-uniform)
@@ -312,18 +340,36 @@ __global__ void __launch_bounds__(NT) inter_kernel(InterArgs a) {
     const int item = s_item;
     if (item >= n_items) break;
     if (item < n_long_items) {
-      // ---------------- long pair: chained strips across the CTA's warps
-      const int qr = item / a.n_long, pidx = item - qr * a.n_long;
-      const QueryDesc d = a.queries[qr];
+      // ---------------- long pair, superstrip k: W chained strips on this CTA's
+      // warps; superstrips k-1 / k+1 of the same pair run on other CTAs
+      int lo = 0, hi = a.n_queries - 1;
+      while (lo < hi) {
+        const int mid = (lo + hi + 1) >> 1;
+        if (a.queries[mid].long_item_begin <= item) lo = mid; else hi = mid - 1;
+      }
+      const QueryDesc d = a.queries[lo];
+      const int K = d.n_super;               // CTAs sharing this pair
+      const int local = item - d.long_item_begin;
+      const int pidx = local / K, c = local - pidx * K;
       const PairRec pr = a.pairs[pidx];
       const int T = pr.len + 32 * SubLanes<LONG_R>::V;
       uint32_t best = 0;
       uint8_t* myprof = lprof + warp * a.SBL;
       uint2* links = a.links + (size_t)blockIdx.x * W * a.lcap;
-      // Upstream strips run on the HIGHER warp ids: the SMSP arbiter issues
-      // highest-warp-id first, so producers keep their lead instead of being
-      // starved by consumers that caught up and spin on the link counter.
-      for (int s = W - 1 - warp; s < d.n_strips_long; s += W) {
+      uint2* grow = a.glinks + d.glink_base + a.lofs[pidx];
+      int* gflag = a.gflags + d.flag_base + (int64_t)pidx * K;
+      // Strips are dealt round-robin: round r of CTA c covers strips
+      // W*(K*r + c) .. +W-1, one per warp.  Upstream strips run on the HIGHER
+      // warp ids: the SMSP arbiter issues highest-warp-id first, so producers
+      // keep their lead instead of being starved by consumers that caught up
+      // and spin on the link counter.  The chain runs warp W-1 -> 0 inside a
+      // CTA, then on to CTA c+1 (global boundary row + GPU-scope counter), and
+      // from CTA K-1 back to CTA 0 for the next round.
+      const int j = W - 1 - warp;
+      const int ns = d.n_strips_long;
+      for (int r = 0;; ++r) {
+        const int s = W * (K * r + c) + j;   // strip index
+        if (s >= ns) break;
         __syncwarp();
         {  // this warp's strip profile -> its own slot
           const uint4* src = reinterpret_cast<const uint4*>(d.prof_long + (size_t)s * a.SBL);
@@ -331,12 +377,32 @@ __global__ void __launch_bounds__(NT) inter_kernel(InterArgs a) {
           for (int i = lane; i < a.SBL / 16; i += 32) dst[i] = __ldg(src + i);
         }
         __syncwarp();
-        const bool rd = s > 0, wr = s + 1 < d.n_strips_long;
-        const int lin = (s + W - 1) % W, lout = s % W;
-        strip_pass<32, LONG_R, true>(myprof, a.LSL, a.LBL, a.stream + pr.off, pr.len, T, lane, rd, wr,
-                                     links + (size_t)lin * a.lcap, links + (size_t)lout * a.lcap,
-                                     &s_prog[lin], (s - 1) << 20, &s_prog[lout], s << 20, a.code_pad2, a.nGe,
-                                     a.nGsGe, best);
+        const bool rd = s > 0, wr = s + 1 < ns;
+        Link lk{};
+        const uint2* rp;
+        uint2* wp;
+        if (j > 0 || K == 1) {  // producer is a warp of this CTA (for K == 1: the last warp, previous round)
+          const int jl = (j + W - 1) % W;
+          rp = links + (size_t)jl * a.lcap;
+          lk.in = &s_prog[jl];
+        } else {                // producer is the last warp of CTA c-1 (or of CTA K-1, previous round)
+          const int pc = (c + K - 1) % K;
+          rp = grow + (int64_t)pc * a.glink_stride;
+          lk.in = gflag + pc;
+          lk.in_gpu = true;
+        }
+        lk.in_base = (s - 1) << 20;  // counters are monotone: (strip << 20) | cells written
+        if (j < W - 1 || K == 1) {
+          wp = links + (size_t)j * a.lcap;
+          lk.out = &s_prog[j];
+        } else {
+          wp = grow + (int64_t)c * a.glink_stride;
+          lk.out = gflag + c;
+          lk.out_gpu = true;
+        }
+        lk.out_base = s << 20;
+        strip_pass<32, LONG_R, true>(myprof, a.LSL, a.LBL, a.stream + pr.off, pr.len, T, lane, rd, wr, rp, wp, lk,
+                                     a.code_pad2, a.nGe, a.nGsGe, best);
       }
 #pragma unroll
       for (int o = 16; o > 0; o >>= 1) best = __vmaxs2(best, __shfl_xor_sync(FULL, best, o));
@@ -345,7 +411,26 @@ __global__ void __launch_bounds__(NT) inter_kernel(InterArgs a) {
       if (tid == 0) {
         uint32_t b = 0;
         for (int w = 0; w < W; ++w) b = __vmaxs2(b, s_best[w]);
-        emit_pair(a, d, pidx, pr, b);
+        if (K == 1) {
+          emit_pair(a, d, pidx, pr, b);
+        } else {  // combine the superstrips' maxima; the last one to finish checks overflow
+          atomicMax(d.scores + pr.id0, int(int16_t(b & 0xffffu)));
+          if (pr.id1 >= 0) atomicMax(d.scores + pr.id1, int(int16_t(b >> 16)));
+          __threadfence();
+          if (atomicAdd(a.gdone + d.done_base + pidx, 1) == K - 1) {
+            __threadfence();
+            const int v0 = atomicAdd(d.scores + pr.id0, 0);
+            const int v1 = pr.id1 >= 0 ? atomicAdd(d.scores + pr.id1, 0) : 0;
+            if (v0 >= a.thr) {
+              const int e = atomicAdd(a.ovf_count, 1);
+              if (e < a.ovf_cap) a.ovf[e] = OvfRec{d.qidx, pidx, 0, 0};
+            }
+            if (pr.id1 >= 0 && v1 >= a.thr) {
+              const int e = atomicAdd(a.ovf_count, 1);
+              if (e < a.ovf_cap) a.ovf[e] = OvfRec{d.qidx, pidx, 1, 0};
+            }
+          }
+        }
       }
     } else {
       // ---------------- short work: find the slot of this item (slots are few)
@@ -386,11 +471,11 @@ __global__ void __launch_bounds__(NT) inter_kernel(InterArgs a) {
         }
         if (q2)
           strip_pass<G, R, false, true>(sprof, a.LS2, a.LB2, a.stream + pr.off, pr.len, T, k, s > 0,
-                                        s + 1 < d.n_strips, bb, bb, nullptr, 0, nullptr, 0, a.code_pad2,
+                                        s + 1 < d.n_strips, bb, bb, Link{}, a.code_pad2,
                                         a.nGe, a.nGsGe, best, half ? 8u : 0u);
         else
           strip_pass<G, R, false>(sprof, a.LS, a.LB, a.stream + pr.off, pr.len, T, k, s > 0, s + 1 < d.n_strips,
-                                  bb, bb, nullptr, 0, nullptr, 0, a.code_pad2, a.nGe, a.nGsGe, best);
+                                  bb, bb, Link{}, a.code_pad2, a.nGe, a.nGsGe, best);
       }
 #pragma unroll
       for (int o = G / 2; o > 0; o >>= 1) best = __vmaxs2(best, __shfl_xor_sync(FULL, best, o, G));
@@ -524,7 +609,9 @@ __global__ void __launch_bounds__(RESCORE_WARPS * 32) rescore_kernel(RescoreArgs
       const int2 z2 = make_int2(0, 0);
       uint2 cw = make_uint2(padw, padw);
       int2 tb0 = z2, tb1 = z2, tb2 = z2, tb3 = z2;
-      if (rd && L > 0) wait_progress(pin, need_base + min(4 + 31 + LINK_LAG, L + 32));
+      const Link lk{const_cast<int*>(pin), need_base, false, const_cast<int*>(pout), pub_base, false};
+      int seen = -1;
+      if (rd && L > 0) wait_progress(lk, need_base + min(4 + 31 + LINK_LAG, L + 32), seen);
       if (lead && L > 0) {
         cw = codes[0];
         if (rd) { tb0 = __ldcg(rp + 0); tb1 = __ldcg(rp + 1); tb2 = __ldcg(rp + 2); tb3 = __ldcg(rp + 3); }
@@ -533,7 +620,7 @@ __global__ void __launch_bounds__(RESCORE_WARPS * 32) rescore_kernel(RescoreArgs
       for (int t0 = 0; t0 < T; t0 += 4) {
         const uint2 cwc = cw;
         const int2 c0 = tb0, c1 = tb1, c2 = tb2, c3 = tb3;
-        if (rd && t0 + 4 < L) wait_progress(pin, need_base + min(t0 + 8 + 31 + LINK_LAG, L + 32));
+        if (rd && t0 + 4 < L) wait_progress(lk, need_base + min(t0 + 8 + 31 + LINK_LAG, L + 32), seen);
         if (lead) {
           if (t0 + 4 < L) {
             cw = codes[(t0 + 4) >> 2];
@@ -578,7 +665,7 @@ __global__ void __launch_bounds__(RESCORE_WARPS * 32) rescore_kernel(RescoreArgs
           sC = rC;
           if (wr && tail) __stcg(wp + t0 + j, make_int2(sH, sF));
         }
-        if (wr && tail) st_release_cta(pout, pub_base + t0 + 4);
+        if (wr && tail) st_release_cta(const_cast<int*>(pout), pub_base + t0 + 4);
       }
     }
 #pragma unroll

@@ -57,7 +57,13 @@ struct QueryDesc {
   const uint8_t* prof_long;  // long-pair (intra-task) profile, [n_strips_long][SBL]
   int32_t* scores;           // this query's row of scores[Q][N] (caller order)
   int n_strips, n_strips_long;
-  int qidx, pad_;
+  int qidx;
+  int n_super;               // superstrips of W = NT/32 strips per long pair
+  int long_item_begin;       // first long work item of this query (n_long * n_super items)
+  int flag_base;             // this query's superstrip counters: gflags[flag_base + pair * n_super + k]
+  int done_base;             // per-pair superstrip completion counters: gdone[done_base + pair]
+  int pad_;
+  int64_t glink_base;        // boundary rows: glinks[glink_base + k * glink_stride + lofs[pair] ...]
 };
 
 // Short-pair work of one "slot": a single query (mode 0: two DB sequences per
@@ -84,8 +90,14 @@ struct InterArgs {
   int SB2, LS2, LB2;         // mode 1 (query-pair) profile
   int SBL, LSL, LBL;         // long geometry (32 lanes x LONG_R rows)
   int n_long;                // pairs [0, n_long) are long (intra-task items)
-  uint2* links;              // [gridDim][NT/32][lcap] strip-to-strip rows (long items)
+  int n_long_items;          // sum over queries of n_long * n_super
+  uint2* links;              // [gridDim][NT/32][lcap] strip-to-strip rows inside a CTA (long items)
   int lcap;
+  uint2* glinks;             // superstrip boundary rows (between CTAs)
+  int* gflags;               // their progress counters (zeroed per search)
+  int* gdone;                // per (query, long pair) superstrip completion counters (zeroed per search)
+  const int64_t* lofs;       // per long pair: offset of its boundary row (sum of (len + 72) before it)
+  int64_t glink_stride;      // sum over long pairs of (len + 72)
   const uint16_t* stream;
   const PairRec* pairs;
   int pair_begin, pair_end;  // [begin, end): the short pairs

@@ -193,11 +193,12 @@ def test_swissprot_scale_sampled(name):
 
 def test_intra_task_mode_forced():
     """t_long small: most pairs go through the chained-warps (intra-task) mode;
-    queries span 1 strip, exactly 1, 2, and more strips than warps (ring wrap)."""
+    queries span 1 strip, 2 strips, and more strips than one CTA's warps (the
+    pair is then split into superstrips chained across CTAs)."""
     rng = np.random.default_rng(21)
     dl = list(rng.integers(1, 700, size=70)) + [0, 1, 65, 66, 67, 68]
     dc, do = _seqs(dl, rng)
-    ql = [1, 100, 256, 257, 600, 2400]
+    ql = [1, 100, 256, 257, 600, 2400, 4100, 13000]   # 13000 rows: the pair is split over 2 CTAs
     qc, qo = _seqs(ql, rng)
     got = gpu_scores(qc, qo, dc, do, opts={"t_long": 64})
     np.testing.assert_array_equal(got, oracle_scores(qc, qo, dc, do))

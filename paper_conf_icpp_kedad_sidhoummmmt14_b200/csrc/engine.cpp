@@ -72,7 +72,10 @@ struct SwError {
 [[noreturn]] void fail(int32_t code, const std::string& m) { throw SwError{code, m}; }
 
 constexpr int T_LONG = 3000;
-constexpr int LONG_ROUNDS = 3;  // target rounds of W strips per CTA for a long pair  // pairs longer than this are launched separately
+constexpr int LONG_ROUNDS = 3;  // target rounds of W strips per CTA for a long pair
+// A short item (one lane group, all strips of its query) may not run longer than
+// this many wavefront steps; pairs beyond it go to the intra-task mode.
+constexpr int64_t CRIT_STEPS = 200000;  // pairs longer than this are launched separately
 
 }  // namespace
 
@@ -87,6 +90,8 @@ struct sw_handle_s {
   // scratch (grown on demand)
   DevBuf qcodes, qoff, matrix, prof, bbuf, bbuf_long, counters, ovf, ovf_count, scores_tmp, rbuf, qdesc;
   DevBuf glinks, gflags;  // superstrip boundary rows and their counters (long pairs)
+  DevBuf rgrows, rflags;  // re-score: CTA-to-CTA rows, counters
+  int* pinned_count = nullptr;
   cudaEvent_t ev_begin = nullptr, ev_end = nullptr;
   bool search_timed = false;
   bool timing_accumulate = false;
@@ -114,8 +119,9 @@ struct sw_db_s {
   // per-DB constants of the pair table (computed once at load)
   double sum_short_len = 0, sum_long_len = 0, short_res = 0;
   int32_t max_short = 0, max_long = 0;
-  int64_t glink_stride = 0;      // sum over long pairs of (len + 72): one superstrip boundary row set
-  DevBuf dlofs;                  // per long pair: offset of its boundary row
+  std::vector<int64_t> lofs_host;   // [np+1] prefix of (len + 72): boundary-row offsets
+  std::vector<int64_t> len_prefix;  // [np+1] prefix of padded pair lengths
+  DevBuf dlofs;
   DevBuf stream, dpairs;
 };
 
@@ -278,13 +284,16 @@ int32_t sw_load_db(sw_handle_t h, const uint8_t* codes, const int64_t* offsets, 
       }
     }
     std::vector<uint16_t>& stream = P.stream;
-    {
-      std::vector<int64_t> lofs(size_t(std::max(db->n_long, 1)), 0);
-      int64_t acc = 0;
-      for (int p = 0; p < db->n_long; ++p) { lofs[size_t(p)] = acc; acc += db->pairs[size_t(p)].len + 72; }
-      db->glink_stride = acc;
-      SW_CK(db->dlofs.ensure(lofs.size() * sizeof(int64_t)));
-      SW_CK(cudaMemcpyAsync(db->dlofs.p, lofs.data(), lofs.size() * sizeof(int64_t), cudaMemcpyHostToDevice, st));
+    {  // boundary-row offsets of every pair (any pair may be a long item for a tall query)
+      db->lofs_host.assign(np + 1, 0);
+      db->len_prefix.assign(np + 1, 0);
+      for (size_t p = 0; p < np; ++p) {
+        db->lofs_host[p + 1] = db->lofs_host[p] + db->pairs[p].len + 72;
+        db->len_prefix[p + 1] = db->len_prefix[p] + db->pairs[p].len;
+      }
+      SW_CK(db->dlofs.ensure(db->lofs_host.size() * sizeof(int64_t)));
+      SW_CK(cudaMemcpyAsync(db->dlofs.p, db->lofs_host.data(), db->lofs_host.size() * sizeof(int64_t),
+                            cudaMemcpyHostToDevice, st));
     }
     SW_CK(db->stream.ensure(stream.size() * sizeof(uint16_t)));
     SW_CK(db->dpairs.ensure(std::max<size_t>(np, 1) * sizeof(PairRec)));
@@ -348,8 +357,6 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
   sw_db_s* db = c.db;
   const int alpha = db->alpha;
   const int np = int(db->pairs.size());
-  const int nlong = db->n_long;
-  const int nshort = np - nlong;
   std::vector<int> order;
   for (int i = 0; i < int(qlen.size()); ++i)
     if (qlen[size_t(i)] > 0) order.push_back(i);
@@ -358,30 +365,52 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
   std::vector<int> ms;
   for (int i : order) ms.push_back(int(qlen[size_t(i)]));
   // short-pair slots: neighbours in length order form query pairs (mode 1)
-  struct Slot { int mode, k0, k1; };
+  struct Slot { int mode, k0, k1, nlong; };
   std::vector<Slot> slots;
   const bool pairs_on = h->opt_query_pairs != 0;
   for (size_t k = 0; k < order.size();) {
-    if (pairs_on && k + 1 < order.size()) { slots.push_back({1, int(k), int(k + 1)}); k += 2; }
-    else { slots.push_back({0, int(k), -1}); k += 1; }
+    if (pairs_on && k + 1 < order.size()) { slots.push_back({1, int(k), int(k + 1), 0}); k += 2; }
+    else { slots.push_back({0, int(k), -1, 0}); k += 1; }
   }
   std::vector<std::pair<int, int>> slot_m;
   for (auto& sl : slots) slot_m.push_back({ms[size_t(sl.k0)], sl.mode});
+  const int nlong_db = db->n_long;  // pairs longer than t_long
+  const int nshort_db = np - nlong_db;
   int G = 4, R = 24;
-  choose_geom(h, slot_m, nshort > 0 ? c.sum_short / nshort : 1.0, G, R);
+  choose_geom(h, slot_m, nshort_db > 0 ? db->sum_short_len / nshort_db : 1.0, G, R);
   if (!inter_config_supported(G, R)) fail(SW_EUNSUPPORTED, "no kernel for this geometry");
   const int NT = inter_block_threads(), NG = NT / G, W = NT / 32;
   const int LB2 = (((R / 4) | 1) * 16);
   const int LS2 = G * LB2;
   const int SB2 = (((alpha + 1) * LS2 + 15) / 16) * 16;
+  // Per slot, pairs [0, nlong) go to the intra-task (long) mode: those longer
+  // than t_long, plus -- for very tall queries -- shorter pairs whose one-group
+  // critical path (strips x columns) would otherwise outlast the search.
+  auto pairs_longer_than = [&](int64_t Lc) {  // pairs are sorted longest first
+    int lo = 0, hi = np;
+    while (lo < hi) { const int mid = (lo + hi) / 2; if (db->pairs[size_t(mid)].len > Lc) lo = mid + 1; else hi = mid; }
+    return lo;
+  };
+  int nlong_max = 0;
+  for (auto& sl : slots) {
+    const int strips = std::max(1, (ms[size_t(sl.k0)] + G * R - 1) / (G * R));
+    const int64_t Lc = std::min<int64_t>(h->opt_t_long, CRIT_STEPS / strips);
+    sl.nlong = std::max(nlong_db, pairs_longer_than(Lc));
+    nlong_max = std::max(nlong_max, sl.nlong);
+  }
+  std::vector<int> qnlong(order.size(), 0);
+  for (auto& sl : slots) {
+    qnlong[size_t(sl.k0)] = sl.nlong;
+    if (sl.k1 >= 0) qnlong[size_t(sl.k1)] = sl.nlong;
+  }
   // profiles: long geometry per query; short geometry per slot
   size_t total = 0;
   std::vector<ProfGeom> gl;
   std::vector<size_t> off_l;
-  for (int m : ms) {
-    gl.push_back(make_geom(32, LONG_R, m, alpha, /*dense=*/true));
+  for (size_t k = 0; k < order.size(); ++k) {
+    gl.push_back(make_geom(32, LONG_R, ms[k], alpha, /*dense=*/true));
     off_l.push_back(total);
-    total += nlong > 0 ? size_t(gl.back().n_strips) * gl.back().SB : 0;
+    total += qnlong[k] > 0 ? size_t(gl.back().n_strips) * gl.back().SB : 0;
   }
   const ProfGeom g1 = make_geom(G, R, 1, alpha);  // SB / LS / LB of the mode-0 profile
   std::vector<size_t> off_s;
@@ -390,20 +419,25 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
     const int n = std::max(1, (ms[size_t(sl.k0)] + G * R - 1) / (G * R));  // k0 is the longer query
     strips_s.push_back(n);
     off_s.push_back(total);
-    if (nshort > 0) total += size_t(n) * (sl.mode == 1 ? SB2 : g1.SB);
+    if (sl.nlong < np) total += size_t(n) * (sl.mode == 1 ? SB2 : g1.SB);
   }
   SW_CK(h->prof.ensure(total + 16));
   uint8_t* prof = h->prof.as<uint8_t>();
   const int8_t* dmat = h->matrix.as<int8_t>();
   auto qptr = [&](int k) { return h->qcodes.as<uint8_t>() + qoff0[size_t(order[size_t(k)])]; };
+  auto pair_len_sum = [&](int p0, int p1) {  // sum of padded pair lengths over [p0, p1)
+    return double(db->len_prefix[size_t(p1)] - db->len_prefix[size_t(p0)]);
+  };
   std::vector<QueryDesc> desc(order.size());
-  int64_t long_items = 0, flags_total = 0, glink_total = 0;
-  const double sumS = db->sum_short_len + double(nshort) * G, sumL = db->sum_long_len + double(nlong) * 32;
+  int64_t long_items = 0, flags_total = 0, glink_total = 0, done_total = 0;
+  int max_lstrips = 1;
   for (size_t k = 0; k < order.size(); ++k) {
     const int qi = order[k];
-    if (nlong > 0) {
+    const int nl = qnlong[k];
+    if (nl > 0) {
       SW_CK(launch_build_profile(qptr(int(k)), ms[k], dmat, alpha, gl[k], prof + off_l[k], c.st));
       ++launches;
+      max_lstrips = std::max(max_lstrips, gl[k].n_strips);
     }
     QueryDesc& d = desc[k];
     d.prof = nullptr;
@@ -412,24 +446,28 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
     d.n_strips = 0;
     d.n_strips_long = gl[k].n_strips;
     d.qidx = qi;
+    d.n_long = nl;
     // CTAs per long pair: enough to split very tall queries, few enough that each
     // CTA still runs ~LONG_ROUNDS rounds of W strips (amortises the pipeline ramp)
     d.n_super = std::max(1, (gl[k].n_strips + W * LONG_ROUNDS - 1) / (W * LONG_ROUNDS));
     d.long_item_begin = int(long_items);
     d.flag_base = int(flags_total);
-    d.done_base = int(k) * nlong;
-    d.pad_ = 0;
+    d.done_base = int(done_total);
     d.glink_base = glink_total;
-    long_items += int64_t(nlong) * d.n_super;
-    flags_total += int64_t(nlong) * d.n_super;
-    if (d.n_super > 1) glink_total += int64_t(d.n_super) * db->glink_stride;
-    cells_computed += 2.0 * sumL * double(gl[k].n_strips) * 32 * LONG_R;
+    d.glink_stride = db->lofs_host[size_t(nl)];
+    long_items += int64_t(nl) * d.n_super;
+    flags_total += int64_t(nl) * d.n_super;
+    done_total += nl;
+    if (d.n_super > 1) glink_total += int64_t(d.n_super) * d.glink_stride;
+    cells_computed += 2.0 * (pair_len_sum(0, nl) + 32.0 * nl) * double(gl[k].n_strips) * 32 * LONG_R;
   }
   std::vector<SlotDesc> sdesc(slots.size());
   int item = 0;
+  int min_pb = np;
   for (size_t j = 0; j < slots.size(); ++j) {
     const Slot& sl = slots[j];
     SlotDesc& d = sdesc[j];
+    const int ns = np - sl.nlong;  // short pairs of this slot
     d.prof = prof + off_s[j];
     d.mode = sl.mode;
     d.n_strips = strips_s[j];
@@ -437,10 +475,13 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
     d.scores0 = c.dscores + int64_t(d.qidx0) * db->n_seqs;
     d.qidx1 = sl.mode == 1 ? order[size_t(sl.k1)] : -1;
     d.scores1 = sl.mode == 1 ? c.dscores + int64_t(d.qidx1) * db->n_seqs : nullptr;
+    d.pair_begin = sl.nlong;
     d.item_begin = item;
-    d.n_items = nshort > 0 ? (sl.mode == 1 ? (2 * nshort + NG - 1) / NG : (nshort + NG - 1) / NG) : 0;
+    d.n_items = ns > 0 ? (sl.mode == 1 ? (2 * ns + NG - 1) / NG : (ns + NG - 1) / NG) : 0;
     item += d.n_items;
-    if (nshort > 0) {
+    if (ns > 0) {
+      min_pb = std::min(min_pb, sl.nlong);
+      const double sumS = pair_len_sum(sl.nlong, np) + double(ns) * 2 * G;
       if (sl.mode == 1) {
         SW_CK(launch_build_profile_q2(qptr(sl.k0), ms[size_t(sl.k0)], qptr(sl.k1), ms[size_t(sl.k1)], dmat, alpha,
                                       G, R, LB2, d.n_strips, SB2, prof + off_s[j], c.st));
@@ -459,26 +500,24 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
   SlotDesc* d_slots = reinterpret_cast<SlotDesc*>(d_desc + desc.size());
   SW_CK(cudaMemcpyAsync(d_desc, desc.data(), desc.size() * sizeof(QueryDesc), cudaMemcpyHostToDevice, c.st));
   SW_CK(cudaMemcpyAsync(d_slots, sdesc.data(), sdesc.size() * sizeof(SlotDesc), cudaMemcpyHostToDevice, c.st));
-  std::vector<ProfGeom> gs;
-  for (size_t j = 0; j < slots.size(); ++j) { ProfGeom x = g1; x.n_strips = strips_s[j]; gs.push_back(x); }
-  const ProfGeom g0 = g1, l0 = gl[0];
-  const int smem = std::max(g0.SB, SB2) + (nlong > 0 ? W * l0.SB : 0);
+  int max_strips = 1;
+  for (int n : strips_s) max_strips = std::max(max_strips, n);
+  const ProfGeom l0 = gl[0];
+  const int smem = std::max(g1.SB, SB2) + (nlong_max > 0 ? W * l0.SB : 0);
   const int occ = inter_max_ctas_per_sm(G, R, NT, smem);
   if (occ <= 0) fail(SW_ECUDA, "inter kernel does not fit on an SM");
   const int64_t n_items = long_items + item;
   if (n_items >= (int64_t(1) << 31)) fail(SW_EUNSUPPORTED, "too many work items");
   const int grid = int(std::max<int64_t>(1, std::min<int64_t>(n_items, int64_t(occ) * h->sms)));
-  int max_strips = 1;
-  for (auto& x : gs) max_strips = std::max(max_strips, x.n_strips);
-  int max_lstrips = 1;
-  for (auto& x : gl) max_lstrips = std::max(max_lstrips, x.n_strips);
-  const int bcap = c.max_short + 2 * G + 8;  // wave width up to 2G sub-lanes
-  if (max_strips > 1 && nshort > 0) SW_CK(h->bbuf.ensure(size_t(grid) * NG * bcap * sizeof(uint2)));
-  const int lcap = c.max_long + 64 + 8;
-  if (nlong > 0 && max_lstrips > 1) SW_CK(h->bbuf_long.ensure(size_t(grid) * W * lcap * sizeof(uint2)));
+  const int32_t max_short = min_pb < np ? db->pairs[size_t(min_pb)].len : 0;
+  const int32_t max_long = db->pairs[0].len;
+  const int bcap = max_short + 2 * G + 8;  // wave width up to 2G sub-lanes
+  if (max_strips > 1 && min_pb < np) SW_CK(h->bbuf.ensure(size_t(grid) * NG * bcap * sizeof(uint2)));
+  const int lcap = max_long + 64 + 8;
+  if (nlong_max > 0 && max_lstrips > 1) SW_CK(h->bbuf_long.ensure(size_t(grid) * W * lcap * sizeof(uint2)));
   SW_CK(h->counters.ensure(sizeof(int)));
   SW_CK(cudaMemsetAsync(h->counters.p, 0, sizeof(int), c.st));
-  const size_t nflags = size_t(std::max<int64_t>(flags_total, 1)), ndone = size_t(std::max<int64_t>(int64_t(order.size()) * nlong, 1));
+  const size_t nflags = size_t(std::max<int64_t>(flags_total, 1)), ndone = size_t(std::max<int64_t>(done_total, 1));
   SW_CK(h->gflags.ensure((nflags + ndone) * sizeof(int)));
   SW_CK(cudaMemsetAsync(h->gflags.p, 0, (nflags + ndone) * sizeof(int), c.st));
   if (glink_total > 0) SW_CK(h->glinks.ensure(size_t(glink_total) * sizeof(uint2)));
@@ -491,26 +530,23 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
   a.SB2 = SB2;
   a.LS2 = LS2;
   a.LB2 = LB2;
-  a.SB = g0.SB;
-  a.LS = g0.LS;
-  a.LB = g0.LB;
+  a.SB = g1.SB;
+  a.LS = g1.LS;
+  a.LB = g1.LB;
   a.SBL = l0.SB;
   a.LSL = l0.LS;
   a.LBL = l0.LB;
-  a.n_long = nlong;
   a.n_long_items = int(long_items);
   a.glinks = glink_total > 0 ? h->glinks.as<uint2>() : nullptr;
   a.gflags = h->gflags.as<int>();
   a.gdone = h->gflags.as<int>() + nflags;
   a.lofs = db->dlofs.as<int64_t>();
-  a.glink_stride = db->glink_stride;
-  a.links = (nlong > 0 && max_lstrips > 1) ? h->bbuf_long.as<uint2>() : nullptr;
+  a.links = (nlong_max > 0 && max_lstrips > 1) ? h->bbuf_long.as<uint2>() : nullptr;
   a.lcap = lcap;
   a.stream = db->stream.as<uint16_t>();
   a.pairs = db->dpairs.as<PairRec>();
-  a.pair_begin = nlong;
   a.pair_end = np;
-  a.bbuf = (max_strips > 1 && nshort > 0) ? h->bbuf.as<uint2>() : nullptr;
+  a.bbuf = (max_strips > 1 && min_pb < np) ? h->bbuf.as<uint2>() : nullptr;
   a.bcap = bcap;
   a.work_counter = h->counters.as<int>();
   a.thr = c.thr;
@@ -638,27 +674,51 @@ int32_t sw_search(sw_handle_t h, const uint8_t* q_codes, const int64_t* q_offset
     const uint8_t* dq = h->qcodes.as<uint8_t>();
     launch_all(lc, qlen, qoff0, cells_computed, launches);
     if (ovf_cap > 0) {
-      const int32_t Lmax = std::max(max_short, max_long);
-      const int grid = std::max(1, std::min<int>(int(ovf_cap), h->sms * 2));  // one CTA per flagged pair
-      const int bcap = Lmax + 32 + 8;
-      SW_CK(h->rbuf.ensure(size_t(grid) * RESCORE_WARPS * bcap * sizeof(int2)));
-      RescoreArgs r{};
-      r.qcodes = dq;
-      r.qoff = h->qoff.as<int64_t>();
-      r.stream = db->stream.as<uint16_t>();
-      r.pairs = db->dpairs.as<PairRec>();
-      r.matrix = h->matrix.as<int8_t>();
-      r.alpha = alpha;
-      r.ovf = h->ovf.as<OvfRec>();
-      r.ovf_count = h->ovf_count.as<int>();
-      r.bbuf = h->rbuf.as<int2>();
-      r.bcap = bcap;
-      r.scores = dscores;
-      r.n_seqs = N;
-      r.Gs = gap_open;
-      r.Ge = gap_extend;
-      SW_CK(launch_rescore(grid, r, st));
-      ++launches;
+      // the flagged list is usually empty or tiny: read its length (one sync,
+      // only for searches whose bounds allow an int16 overflow at all)
+      if (!h->pinned_count) SW_CK(cudaMallocHost(&h->pinned_count, sizeof(int)));
+      SW_CK(cudaMemcpyAsync(h->pinned_count, h->ovf_count.p, sizeof(int), cudaMemcpyDeviceToHost, st));
+      SW_CK(cudaStreamSynchronize(st));
+      const int cnt = int(std::min<int64_t>(*h->pinned_count, ovf_cap));
+      if (cnt > 0) {
+        const int32_t Lmax = std::max(max_short, max_long);
+        int64_t mmax = 1;
+        for (auto L : qlen) mmax = std::max(mmax, L);
+        const int rows_per_strip = 32 * RESCORE_R;
+        const int nstrips = int((mmax + rows_per_strip - 1) / rows_per_strip);
+        const int K = std::max(1, (nstrips + RESCORE_WARPS * LONG_ROUNDS - 1) / (RESCORE_WARPS * LONG_ROUNDS));
+        const int grid = std::max(1, std::min<int>(cnt * K, h->sms * 2));
+        const int bcap = Lmax + 32 + 72;
+        SW_CK(h->rbuf.ensure(size_t(grid) * RESCORE_WARPS * bcap * sizeof(int2)));
+        SW_CK(h->rgrows.ensure(size_t(cnt) * K * bcap * sizeof(int2) + 16));
+        const size_t nint = size_t(cnt) * K + 2 * size_t(cnt) + 1;
+        SW_CK(h->rflags.ensure(nint * sizeof(int)));
+        SW_CK(cudaMemsetAsync(h->rflags.p, 0, nint * sizeof(int), st));
+        int* fl = h->rflags.as<int>();
+        RescoreArgs r{};
+        r.qcodes = dq;
+        r.qoff = h->qoff.as<int64_t>();
+        r.stream = db->stream.as<uint16_t>();
+        r.pairs = db->dpairs.as<PairRec>();
+        r.matrix = h->matrix.as<int8_t>();
+        r.alpha = alpha;
+        r.ovf = h->ovf.as<OvfRec>();
+        r.n_entries = cnt;
+        r.K = K;
+        r.gflags = fl;
+        r.acc = fl + size_t(cnt) * K;
+        r.done = r.acc + cnt;
+        r.work_counter = r.done + cnt;
+        r.bbuf = h->rbuf.as<int2>();
+        r.grows = h->rgrows.as<int2>();
+        r.bcap = bcap;
+        r.scores = dscores;
+        r.n_seqs = N;
+        r.Gs = gap_open;
+        r.Ge = gap_extend;
+        SW_CK(launch_rescore(grid, r, st));
+        ++launches;
+      }
     }
     if (timing) {
       SW_CK(cudaEventRecord(h->ev_end, st));
@@ -734,6 +794,7 @@ int32_t sw_free(sw_handle_t h) {
   }
   for (cudaEvent_t e : {h->ev_begin, h->ev_end})
     if (e) cudaEventDestroy(e);
+  if (h->pinned_count) cudaFreeHost(h->pinned_count);
   delete h;
   return SW_OK;
 }

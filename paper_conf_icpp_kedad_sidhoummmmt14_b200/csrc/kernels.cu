@@ -349,6 +349,7 @@ __global__ void __launch_bounds__(NT) inter_kernel(InterArgs a) {
       }
       const QueryDesc d = a.queries[lo];
       const int K = d.n_super;               // CTAs sharing this pair
+      const int64_t gstride = d.glink_stride;
       const int local = item - d.long_item_begin;
       const int pidx = local / K, c = local - pidx * K;
       const PairRec pr = a.pairs[pidx];
@@ -387,7 +388,7 @@ __global__ void __launch_bounds__(NT) inter_kernel(InterArgs a) {
           lk.in = &s_prog[jl];
         } else {                // producer is the last warp of CTA c-1 (or of CTA K-1, previous round)
           const int pc = (c + K - 1) % K;
-          rp = grow + (int64_t)pc * a.glink_stride;
+          rp = grow + (int64_t)pc * gstride;
           lk.in = gflag + pc;
           lk.in_gpu = true;
         }
@@ -396,7 +397,7 @@ __global__ void __launch_bounds__(NT) inter_kernel(InterArgs a) {
           wp = links + (size_t)j * a.lcap;
           lk.out = &s_prog[j];
         } else {
-          wp = grow + (int64_t)c * a.glink_stride;
+          wp = grow + (int64_t)c * gstride;
           lk.out = gflag + c;
           lk.out_gpu = true;
         }
@@ -447,10 +448,10 @@ __global__ void __launch_bounds__(NT) inter_kernel(InterArgs a) {
       int p, half = 0;
       if (q2) {  // chunk of NG half-pairs: DB sequence = one half of a pair
         const int hp = chunk * NG + g;
-        p = a.pair_begin + (hp >> 1);
+        p = d.pair_begin + (hp >> 1);
         half = hp & 1;
       } else {
-        p = a.pair_begin + chunk * NG + g;
+        p = d.pair_begin + chunk * NG + g;
       }
       bool valid = p < a.pair_end;
       PairRec pr;
@@ -551,12 +552,13 @@ cudaError_t launch_inter(int G, int R, int NT, int grid, int smem_bytes, const I
 }
 
 // ---------------------------------------------------------------------------
-// Exact int32 re-score of flagged pairs.  One CTA per pair,
-// the same chained-warp intra-task wavefront as the long-pair mode but one
-// problem per lane in int32 (s32 DPX) and S read from a shared 33x33 matrix:
-// warp w does strips w, w+W, ... (32 lanes x RESCORE_R rows), strip s+1
-// consuming strip s's bottom row through a global link row + shared progress
-// counter.  Codes and link cells are fetched a 4-column block ahead.
+// Exact int32 re-score of flagged pairs.  The same chained
+// wavefront as the long-pair mode, one problem per lane in int32 (s32 DPX),
+// S read from a shared 33x33 matrix: a flagged pair is split over K CTAs,
+// strips dealt round-robin (round r of CTA c = strips W*(K*r + c) .. +W-1,
+// 32 lanes x RESCORE_R rows each), chained warp to warp through per-CTA link
+// rows + shared counters and CTA to CTA through global rows + GPU-scope
+// counters.  The CTAs' maxima meet in acc[e]; the last CTA writes the score.
 __global__ void __launch_bounds__(RESCORE_WARPS * 32) rescore_kernel(RescoreArgs a) {
   constexpr int R = RESCORE_R;
   constexpr int W = RESCORE_WARPS;
@@ -564,6 +566,7 @@ __global__ void __launch_bounds__(RESCORE_WARPS * 32) rescore_kernel(RescoreArgs
   __shared__ int32_t sm[SW * SW];
   __shared__ int s_prog[W];
   __shared__ int s_best[W];
+  __shared__ int s_item;
   for (int i = threadIdx.x; i < SW * SW; i += blockDim.x) {
     const int x = i / SW, y = i % SW;
     sm[i] = (x < a.alpha && y < a.alpha) ? int(a.matrix[x * a.alpha + y]) : int(PAD_SCORE);
@@ -571,13 +574,18 @@ __global__ void __launch_bounds__(RESCORE_WARPS * 32) rescore_kernel(RescoreArgs
   const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
   const bool lead = lane == 0, tail = lane == 31;
   int2* __restrict__ links = a.bbuf + (size_t)blockIdx.x * W * a.bcap;
-  const int cnt = *a.ovf_count;
+  const int K = a.K;
+  const int n_items = a.n_entries * K;
   const int pad = a.alpha;
   const int nGe = -a.Ge, nGsGe = -(a.Gs + a.Ge);
-  for (int e = blockIdx.x; e < cnt; e += gridDim.x) {
+  for (;;) {
     __syncthreads();
+    if (threadIdx.x == 0) s_item = atomicAdd(a.work_counter, 1);
     if (threadIdx.x < W) { s_prog[threadIdx.x] = -1; s_best[threadIdx.x] = 0; }
     __syncthreads();
+    const int item = s_item;
+    if (item >= n_items) break;
+    const int e = item / K, c = item - e * K;
     const OvfRec o = a.ovf[e];
     const PairRec pr = a.pairs[o.pair];
     const uint8_t* qc = a.qcodes + a.qoff[o.q];
@@ -588,30 +596,52 @@ __global__ void __launch_bounds__(RESCORE_WARPS * 32) rescore_kernel(RescoreArgs
     const int T = L + 32;
     const uint2* __restrict__ codes = reinterpret_cast<const uint2*>(a.stream + pr.off);
     const uint32_t padw = uint32_t(pad) * 0x01010101u;
+    int2* grow = a.grows + (int64_t)e * K * a.bcap;
+    int* gflag = a.gflags + (int64_t)e * K;
+    const int j = W - 1 - warp;  // producers on higher warp ids (see inter_kernel)
     int best = 0;
-    for (int s = W - 1 - warp; s < nstrips; s += W) {  // producers on higher warp ids (see inter_kernel)
+    for (int r = 0;; ++r) {
+      const int s = W * (K * r + c) + j;
+      if (s >= nstrips) break;
       const bool rd = s > 0, wr = s + 1 < nstrips;
-      const int lin = (s + W - 1) % W, lout = s % W;
-      const int2* __restrict__ rp = links + (size_t)lin * a.bcap + 31;
-      int2* __restrict__ wp = links + (size_t)lout * a.bcap;
-      volatile int* pin = &s_prog[lin];
-      volatile int* pout = &s_prog[lout];
-      const int need_base = (s - 1) << 20, pub_base = s << 20;
+      Link lk{};
+      const int2* rp;
+      int2* wp;
+      if (j > 0 || K == 1) {
+        const int jl = (j + W - 1) % W;
+        rp = links + (size_t)jl * a.bcap;
+        lk.in = &s_prog[jl];
+      } else {
+        const int pc = (c + K - 1) % K;
+        rp = grow + (int64_t)pc * a.bcap;
+        lk.in = gflag + pc;
+        lk.in_gpu = true;
+      }
+      lk.in_base = (s - 1) << 20;
+      if (j < W - 1 || K == 1) {
+        wp = links + (size_t)j * a.bcap;
+        lk.out = &s_prog[j];
+      } else {
+        wp = grow + (int64_t)c * a.bcap;
+        lk.out = gflag + c;
+        lk.out_gpu = true;
+      }
+      lk.out_base = s << 20;
+      rp += 31;
       int qr[R], Hl[R], E[R];
 #pragma unroll
-      for (int r = 0; r < R; ++r) {
-        const int row = s * 32 * R + lane * R + r;
-        qr[r] = (row < m ? int(qc[row]) : pad) * SW;
-        Hl[r] = 0;
-        E[r] = 0;
+      for (int rr = 0; rr < R; ++rr) {
+        const int row = s * 32 * R + lane * R + rr;
+        qr[rr] = (row < m ? int(qc[row]) : pad) * SW;
+        Hl[rr] = 0;
+        E[rr] = 0;
       }
       int hdiag = 0, sH = 0, sF = 0, sC = pad;
       const int2 z2 = make_int2(0, 0);
       uint2 cw = make_uint2(padw, padw);
       int2 tb0 = z2, tb1 = z2, tb2 = z2, tb3 = z2;
-      const Link lk{const_cast<int*>(pin), need_base, false, const_cast<int*>(pout), pub_base, false};
       int seen = -1;
-      if (rd && L > 0) wait_progress(lk, need_base + min(4 + 31 + LINK_LAG, L + 32), seen);
+      if (rd && L > 0) wait_progress(lk, lk.in_base + min(4 + 31 + LINK_LAG, L + 32), seen);
       if (lead && L > 0) {
         cw = codes[0];
         if (rd) { tb0 = __ldcg(rp + 0); tb1 = __ldcg(rp + 1); tb2 = __ldcg(rp + 2); tb3 = __ldcg(rp + 3); }
@@ -620,7 +650,7 @@ __global__ void __launch_bounds__(RESCORE_WARPS * 32) rescore_kernel(RescoreArgs
       for (int t0 = 0; t0 < T; t0 += 4) {
         const uint2 cwc = cw;
         const int2 c0 = tb0, c1 = tb1, c2 = tb2, c3 = tb3;
-        if (rd && t0 + 4 < L) wait_progress(lk, need_base + min(t0 + 8 + 31 + LINK_LAG, L + 32), seen);
+        if (rd && t0 + 4 < L) wait_progress(lk, lk.in_base + min(t0 + 8 + 31 + LINK_LAG, L + 32), seen);
         if (lead) {
           if (t0 + 4 < L) {
             cw = codes[(t0 + 4) >> 2];
@@ -634,38 +664,42 @@ __global__ void __launch_bounds__(RESCORE_WARPS * 32) rescore_kernel(RescoreArgs
         }
         __syncwarp();
 #pragma unroll
-        for (int j = 0; j < 4; ++j) {
+        for (int jj = 0; jj < 4; ++jj) {
           int rH = __shfl_up_sync(FULL, sH, 1);
           int rF = __shfl_up_sync(FULL, sF, 1);
           int rC = __shfl_up_sync(FULL, sC, 1);
           if (lead) {
-            const uint32_t w = (j < 2) ? cwc.x : cwc.y;
-            rC = int(((j & 1) ? (w >> 16) : w) >> shift) & 0xff;
-            const int2 tv = (j == 0) ? c0 : (j == 1) ? c1 : (j == 2) ? c2 : c3;
+            const uint32_t w = (jj < 2) ? cwc.x : cwc.y;
+            rC = int(((jj & 1) ? (w >> 16) : w) >> shift) & 0xff;
+            const int2 tv = (jj == 0) ? c0 : (jj == 1) ? c1 : (jj == 2) ? c2 : c3;
             rH = tv.x;
             rF = tv.y;
           }
           int hd = hdiag;
           hdiag = rH;
           int F = rF;
-          int hprev = 0;
+          int dprev = 0;
 #pragma unroll
-          for (int r = 0; r < R; ++r) {
-            const int h = max(__viaddmax_s32(hd, sm[qr[r] + rC], E[r]), F);  // Eq. (2) (E, F >= 0)
-            hd = Hl[r];
-            Hl[r] = h;
+          for (int rr = 0; rr < R; ++rr) {
+            const int dg = hd + sm[qr[rr] + rC];                        // FMA pipe
+            const int h = __vimax3_s32(dg, E[rr], F);                    // Eq. (2) (E, F >= 0)
+            hd = Hl[rr];
+            Hl[rr] = h;
             const int tt = h + nGsGe;
-            E[r] = __viaddmax_s32_relu(E[r], nGe, tt);                               // Eq. (3)
-            F = __viaddmax_s32_relu(F, nGe, tt);                                     // Eq. (4)
-            if (r & 1) best = __vimax3_s32(best, hprev, h);
-            else hprev = h;
+            E[rr] = __viaddmax_s32_relu(E[rr], nGe, tt);                 // Eq. (3)
+            F = __viaddmax_s32_relu(F, nGe, tt);                         // Eq. (4)
+            if (rr & 1) best = __vimax3_s32(best, dprev, dg);            // max D = max H
+            else dprev = dg;
           }
           sH = Hl[R - 1];
           sF = F;
           sC = rC;
-          if (wr && tail) __stcg(wp + t0 + j, make_int2(sH, sF));
+          if (wr && tail) __stcg(wp + t0 + jj, make_int2(sH, sF));
         }
-        if (wr && tail) st_release_cta(const_cast<int*>(pout), pub_base + t0 + 4);
+        if (wr && tail) {
+          if (!lk.out_gpu) st_release_cta(lk.out, lk.out_base + t0 + 4);
+          else if (((t0 >> 2) & 3) == 3 || t0 + 4 >= T) st_release_gpu(lk.out, lk.out_base + t0 + 4);
+        }
       }
     }
 #pragma unroll
@@ -676,13 +710,22 @@ __global__ void __launch_bounds__(RESCORE_WARPS * 32) rescore_kernel(RescoreArgs
       int b = 0;
       for (int w = 0; w < W; ++w) b = max(b, s_best[w]);
       const int id = o.half ? pr.id1 : pr.id0;
-      a.scores[(int64_t)o.q * a.n_seqs + id] = b;
+      if (K == 1) {
+        a.scores[(int64_t)o.q * a.n_seqs + id] = b;
+      } else {
+        atomicMax(a.acc + e, b);
+        __threadfence();
+        if (atomicAdd(a.done + e, 1) == K - 1) {
+          __threadfence();
+          a.scores[(int64_t)o.q * a.n_seqs + id] = atomicAdd(a.acc + e, 0);
+        }
+      }
     }
   }
 }
 
 cudaError_t launch_rescore(int grid, const RescoreArgs& a, cudaStream_t st) {
-  rescore_kernel<<<grid, RESCORE_WARPS * 32, 0, st>>>(a);  // one CTA per flagged pair
+  rescore_kernel<<<grid, RESCORE_WARPS * 32, 0, st>>>(a);  // persistent; K CTAs per flagged pair
   return cudaGetLastError();
 }
 

@@ -62,8 +62,9 @@ struct QueryDesc {
   int long_item_begin;       // first long work item of this query (n_long * n_super items)
   int flag_base;             // this query's superstrip counters: gflags[flag_base + pair * n_super + k]
   int done_base;             // per-pair superstrip completion counters: gdone[done_base + pair]
-  int pad_;
-  int64_t glink_base;        // boundary rows: glinks[glink_base + k * glink_stride + lofs[pair] ...]
+  int n_long;                // pairs [0, n_long) are this query's long items
+  int64_t glink_base;        // boundary rows: glinks[glink_base + c * glink_stride + lofs[pair] ...]
+  int64_t glink_stride;      // sum over this query's long pairs of (len + 72)
 };
 
 // Short-pair work of one "slot": a single query (mode 0: two DB sequences per
@@ -78,6 +79,8 @@ struct SlotDesc {
   int qidx0, qidx1;
   int item_begin;            // first short work item of this slot
   int n_items;               // short work items of this slot
+  int pair_begin;            // short pairs of this slot: [pair_begin, pair_end)
+  int pad_;
 };
 
 struct InterArgs {
@@ -89,18 +92,16 @@ struct InterArgs {
   int SB, LS, LB;            // short geometry (G, R of the launch), mode 0 profile
   int SB2, LS2, LB2;         // mode 1 (query-pair) profile
   int SBL, LSL, LBL;         // long geometry (32 lanes x LONG_R rows)
-  int n_long;                // pairs [0, n_long) are long (intra-task items)
   int n_long_items;          // sum over queries of n_long * n_super
   uint2* links;              // [gridDim][NT/32][lcap] strip-to-strip rows inside a CTA (long items)
   int lcap;
   uint2* glinks;             // superstrip boundary rows (between CTAs)
   int* gflags;               // their progress counters (zeroed per search)
   int* gdone;                // per (query, long pair) superstrip completion counters (zeroed per search)
-  const int64_t* lofs;       // per long pair: offset of its boundary row (sum of (len + 72) before it)
-  int64_t glink_stride;      // sum over long pairs of (len + 72)
+  const int64_t* lofs;       // per pair: offset of its boundary row (sum of (len + 72) before it)
   const uint16_t* stream;
   const PairRec* pairs;
-  int pair_begin, pair_end;  // [begin, end): the short pairs
+  int pair_end;              // number of pairs
   uint2* bbuf;               // boundary rows of multi-strip short items, [gridDim][NG][bcap]
   int bcap;
   int* work_counter;
@@ -119,9 +120,15 @@ struct RescoreArgs {
   const PairRec* pairs;
   const int8_t* matrix;      // alpha x alpha
   int alpha;
-  const OvfRec* ovf;
-  const int* ovf_count;
-  int2* bbuf;                // link rows, [gridDim][RESCORE_WARPS][bcap]
+  const OvfRec* ovf;         // flagged pairs
+  int n_entries;             // number of flagged pairs (host-read count)
+  int K;                     // CTAs per flagged pair
+  int* work_counter;         // zeroed
+  int2* bbuf;                // per-CTA link rows, [gridDim][RESCORE_WARPS][bcap]
+  int2* grows;               // CTA-to-CTA rows, [n_entries][K][bcap]
+  int* gflags;               // [n_entries][K], zeroed
+  int* acc;                  // [n_entries] partial maxima, zeroed
+  int* done;                 // [n_entries] finished CTAs, zeroed
   int bcap;
   int32_t* scores;           // [nq][n_seqs]
   int64_t n_seqs;

@@ -327,11 +327,16 @@ def run_ours(args):
     n_sm = torch.cuda.get_device_properties(dev).multi_processor_count
     peak = n_sm * ALU_LANES_PER_SM_CLK * sm_max * 1e6 / OPS_PER_CELL / 1e9
     achieved = cells_short_step * args.steps / (st["short_ms"] / 1e3) / 1e9 if st["short_ms"] > 0 else None
+    # algorithmic bytes of one launch: every query (pair) pass streams the packed DB once
+    # (~1 B per residue) and the int32 score matrix is written once
+    n_pass = (Q + 1) // 2 if Q > 1 else 1
+    alg_bytes = int(n_pass * int(d_lens.sum()) + 4 * Q * N)
     traffic = None
     tpath = os.path.join(ROOT, "profiles", "traffic.json")
     if os.path.exists(tpath):
         try:
-            traffic = json.load(open(tpath)).get(args.workload)
+            t = json.load(open(tpath)).get(args.workload)
+            traffic = t.get("traffic_bytes_per_launch") if t else None
         except Exception:
             traffic = None
 
@@ -395,6 +400,8 @@ def run_ours(args):
                 "roofline": {"bound": "alu", "achieved": round(achieved, 1) if achieved else None,
                              "peak": round(peak, 1), "unit": "GCUPS", "frac": round(achieved / peak, 4) if achieved else None,
                              "traffic": traffic,
+                             "traffic_unit": "DRAM bytes per launch of the scoring kernel (profiles/traffic.json, ncu)",
+                             "algorithmic_bytes_per_launch": alg_bytes,
                              "kernel": "inter_kernel (short pairs), CUDA events around each launch",
                              "peak_basis": f"{n_sm} SMs x {ALU_LANES_PER_SM_CLK} ALU-pipe lanes/clk x {sm_max:.0f} MHz / "
                                            f"{OPS_PER_CELL} ALU lane-ops per cell (minimal s16x2 Gotoh update; "

@@ -8,7 +8,8 @@ import ctypes
 import os
 
 _HERE = os.path.dirname(os.path.abspath(__file__))
-LIB_PATH = os.path.join(_HERE, "libswdual.so")
+# SWDUAL_LIB overrides the in-tree library (A/B experiments with alternative builds)
+LIB_PATH = os.environ.get("SWDUAL_LIB") or os.path.join(_HERE, "libswdual.so")
 
 SW_OK, SW_EINVAL, SW_ENOMEM, SW_ECUDA, SW_ESTATE, SW_EUNSUPPORTED = 0, -1, -2, -3, -4, -5
 SW_FLAG_TIMING = 1

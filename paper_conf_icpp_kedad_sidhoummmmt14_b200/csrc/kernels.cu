@@ -203,7 +203,7 @@ __device__ __forceinline__ void strip_pass(const uint8_t* sprof, int LS, int LB,
   int seen = -1;
   if (LINKED && rd && L > 0) wait_progress(lk, lk.in_base + min(4 + VG - 1 + LINK_LAG, L + VG), seen);
   if (lead && L > 0) {
-    cw = codes[0];
+    cw = __ldcs(codes);
     if (rd) {
       if (LINKED) { tb0 = __ldcg(rp + 0); tb1 = __ldcg(rp + 1); tb2 = __ldcg(rp + 2); tb3 = __ldcg(rp + 3); }
       else { tb0 = rp[0]; tb1 = rp[1]; tb2 = rp[2]; tb3 = rp[3]; }
@@ -217,7 +217,7 @@ __device__ __forceinline__ void strip_pass(const uint8_t* sprof, int LS, int LB,
     if (LINKED && rd && t0 + 4 < L) wait_progress(lk, lk.in_base + min(t0 + 8 + VG - 1 + LINK_LAG, L + VG), seen);
     if (lead) {
       if (t0 + 4 < L) {
-        cw = codes[(t0 + 4) >> 2];
+        cw = __ldcs(codes + ((t0 + 4) >> 2));
         if (rd) {
           if (LINKED) { tb0 = __ldcg(rp + 0); tb1 = __ldcg(rp + 1); tb2 = __ldcg(rp + 2); tb3 = __ldcg(rp + 3); }
           else { tb0 = rp[0]; tb1 = rp[1]; tb2 = rp[2]; tb3 = rp[3]; }

@@ -64,6 +64,7 @@ def parse():
     ap.add_argument("--e2e-steps", type=int, default=2)
     ap.add_argument("--no-cpu-baseline", action="store_true")
     ap.add_argument("--cpu-baseline-cells", type=float, default=3.0e10)
+    ap.add_argument("--force-geom", default=None, help="G,R of the inter-task kernel (experiments; default auto)")
     ap.add_argument("--verify", type=int, default=0, help="after timing, check N sampled DB sequences "
                     "of the assembled scores against the CPU oracle (rank 0)")
     ap.add_argument("--dist-backend", default="nccl", help="nccl (default); gloo only for functional checks "
@@ -248,6 +249,10 @@ def run_ours(args):
 
     S = sw.blosum62()
     h = sw.Handle(local, timing=True)
+    if args.force_geom:
+        fg, fr = (int(x) for x in args.force_geom.split(","))
+        h.set_option("force_G", fg)
+        h.set_option("force_R", fr)
     dbs = {}
     for s, _qs in blocks:
         sc, so = swdist.subset(c["dcodes"], c["doff"], shards[s])

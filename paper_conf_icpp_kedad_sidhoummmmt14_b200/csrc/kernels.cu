@@ -167,35 +167,10 @@ __device__ __forceinline__ void copy_strip(uint8_t* dst, const uint8_t* __restri
 // its progress counter, lane G-1 publishes its own.
 template <int R>
 struct SubLanes {
-  // Each lane runs V "sub-lanes" of R/V rows, sub-lane u one column behind
-  // sub-lane u-1: V independent dependency chains per step (V times the ILP of
-  // the row-to-row F chain), at the cost of a (V*G - 1)-column wave fill.
-  static constexpr int V = (R % 8 == 0) ? 2 : 1;  // V = 3 measured slower (registers, moves)
-};
-
-// Sub-lanes u = V-1 .. 1 of one step: each takes the previous step's outputs of
-// sub-lane u-1 (carried in registers) and computes its rows one column behind.
-template <int R, int V, int U, bool Q2>
-struct SubStep {
-  __device__ __forceinline__ static void run(const uint32_t (&Hin)[R], uint32_t (&Hout)[R], uint32_t (&E)[R],
-                                             uint32_t& best, uint32_t (&hd)[V], uint32_t (&cH)[V],
-                                             uint32_t (&cF)[V], const uint8_t* (&cpa)[V],
-                                             const uint8_t* (&cpb)[V], uint32_t (&oH)[V], uint32_t (&oF)[V],
-                                             uint32_t nGe, uint32_t nGsGe) {
-    constexpr int RH = R / V;
-    uint32_t h = cH[U], f = cF[U];
-    gotoh_rows<R, U * RH, (U + 1) * RH, Q2>(Hin, Hout, E, best, hd[U], cpa[U], cpb[U], h, f, nGe, nGsGe);
-    oH[U] = h;
-    oF[U] = f;
-    SubStep<R, V, U - 1, Q2>::run(Hin, Hout, E, best, hd, cH, cF, cpa, cpb, oH, oF, nGe, nGsGe);
-  }
-};
-template <int R, int V, bool Q2>
-struct SubStep<R, V, 0, Q2> {
-  __device__ __forceinline__ static void run(const uint32_t (&)[R], uint32_t (&)[R], uint32_t (&)[R], uint32_t&,
-                                             uint32_t (&)[V], uint32_t (&)[V], uint32_t (&)[V],
-                                             const uint8_t* (&)[V], const uint8_t* (&)[V], uint32_t (&)[V],
-                                             uint32_t (&)[V], uint32_t, uint32_t) {}
+  // Each lane runs V "sub-lanes" of R/V rows, the second one column behind the
+  // first: two independent dependency chains per step (twice the ILP of the
+  // row-to-row F chain), at the cost of a (V*G - 1)-column wave fill.
+  static constexpr int V = (R % 8 == 0) ? 2 : 1;
 };
 
 template <int G, int R, bool LINKED, bool Q2 = false>
@@ -215,16 +190,10 @@ __device__ __forceinline__ void strip_pass(const uint8_t* sprof, int LS, int LB,
   const uint32_t laneoff = uint32_t(k) * LB;
   const bool lead = (k == 0), tail = (k == G - 1);
   const uint2 z2 = make_uint2(0, 0);
-  // sub-lanes u >= 1: their inputs are sub-lane u-1's outputs of the previous step
-  uint32_t hdv[V], cH[V], cF[V], cC[V], oH[V], oF[V];
+  // second sub-lane: its inputs are the first sub-lane's outputs of the previous step
+  uint32_t hdiag1 = 0, cH = 0, cF = 0, pC = code_pad2;
   const uint8_t* pad_row = sprof + (code_pad2 & 0xffu) * LS + laneoff;
-  const uint8_t* cpa[V];
-  const uint8_t* cpb[V];
-#pragma unroll
-  for (int u = 0; u < V; ++u) {
-    hdv[u] = 0; cH[u] = 0; cF[u] = 0; cC[u] = code_pad2; oH[u] = 0; oF[u] = 0;
-    cpa[u] = pad_row; cpb[u] = pad_row;
-  }
+  const uint8_t *ppa = pad_row, *ppb = pad_row;
   rp += VG - 1;  // sub-lane 0 of lane 0 reads column c at rp[c + VG - 1]
 
   // lane 0 prefetch of block 0: 4 columns of codes and (if rd) 4 boundary cells.
@@ -281,23 +250,23 @@ __device__ __forceinline__ void strip_pass(const uint8_t* sprof, int LS, int LB,
         pb = sprof + (rC >> 8) * LS + laneoff;
       }
       // even steps read HA and write HB, odd steps the reverse (4 steps per block)
-      if constexpr (V >= 2) {
+      if constexpr (V == 2) {
+        uint32_t h1 = cH, f1 = cF;
         if (j & 1) {
-          SubStep<R, V, V - 1, Q2>::run(HB, HA, E, best, hdv, cH, cF, cpa, cpb, oH, oF, nGe, nGsGe);
+          gotoh_rows<R, RH, R, Q2>(HB, HA, E, best, hdiag1, ppa, ppb, h1, f1, nGe, nGsGe);
           gotoh_rows<R, 0, RH, Q2>(HB, HA, E, best, hdiag, pa, pb, rH, rF, nGe, nGsGe);
         } else {
-          SubStep<R, V, V - 1, Q2>::run(HA, HB, E, best, hdv, cH, cF, cpa, cpb, oH, oF, nGe, nGsGe);
+          gotoh_rows<R, RH, R, Q2>(HA, HB, E, best, hdiag1, ppa, ppb, h1, f1, nGe, nGsGe);
           gotoh_rows<R, 0, RH, Q2>(HA, HB, E, best, hdiag, pa, pb, rH, rF, nGe, nGsGe);
         }
-        // the last sub-lane feeds the next lane; every other output moves one sub-lane down
-        sH = oH[V - 1];
-        sF = oF[V - 1];
-        sC = cC[V - 1];
-#pragma unroll
-        for (int u = V - 1; u >= 2; --u) {
-          cH[u] = oH[u - 1]; cF[u] = oF[u - 1]; cC[u] = cC[u - 1]; cpa[u] = cpa[u - 1]; cpb[u] = cpb[u - 1];
-        }
-        cH[1] = rH; cF[1] = rF; cC[1] = rC; cpa[1] = pa; cpb[1] = pb;
+        cH = rH;
+        cF = rF;
+        ppa = pa;
+        ppb = pb;
+        sH = h1;
+        sF = f1;
+        sC = pC;
+        pC = rC;
       } else {
         if (j & 1) gotoh_rows<R, 0, R, Q2>(HB, HA, E, best, hdiag, pa, pb, rH, rF, nGe, nGsGe);
         else gotoh_rows<R, 0, R, Q2>(HA, HB, E, best, hdiag, pa, pb, rH, rF, nGe, nGsGe);

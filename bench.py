@@ -249,6 +249,9 @@ def run_ours(args):
 
     S = sw.blosum62()
     h = sw.Handle(local, timing=True)
+    for kv in filter(None, os.environ.get("SWDUAL_OPTS", "").split(",")):
+        k_, v_ = kv.split("=")
+        h.set_option(k_, int(v_))
     if args.force_geom:
         fg, fr = (int(x) for x in args.force_geom.split(","))
         h.set_option("force_G", fg)

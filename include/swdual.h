@@ -126,9 +126,13 @@ int32_t sw_last_stats(sw_handle_t h, sw_stats_t* out);
  *   "force_G", "force_R"  force the inter-task lane-group geometry (0 = auto)
  *   "query_pairs"         1 (default): queries are paired two per s16x2 register for
  *                         the short DB pairs (no PRMT); 0: one query per register
- *   "t_long"              DB pairs longer than this (default 3000) are scored in
- *                         the intra-task mode (all warps of a CTA on one pair);
- *                         applies to databases loaded afterwards
+ *   "t_long"              >= 0: DB pairs longer than this are always scored in the
+ *                         intra-task mode (whole CTAs on one pair); default -1:
+ *                         automatic (pairs whose one-lane-group critical path
+ *                         would outlast the search's average share, and every
+ *                         pair > 3000 when such pairs hold most of the residues)
+ *   "pack_long"           1: pack several long pairs per CTA when a query has
+ *                         fewer intra-task strips than warps (default 0)
  *   "timing"              1/0, same as SW_FLAG_TIMING
  *   "timing_accumulate"   1: short_ms/long_ms of sw_last_stats sum every search
  *                         since the last "timing_reset" (0: the last search only)

@@ -73,9 +73,11 @@ struct SwError {
 
 constexpr int T_LONG = 3000;
 constexpr int LONG_ROUNDS = 3;  // target rounds of W strips per CTA for a long pair
-// A short item (one lane group, all strips of its query) may not run longer than
-// this many wavefront steps; pairs beyond it go to the intra-task mode.
-constexpr int64_t CRIT_STEPS = 200000;  // pairs longer than this are launched separately
+// A short item (one lane group, all strips of its query) may run at most
+// max(CRIT_MIN_STEPS, CRIT_FRACTION x the average lane group's wavefront steps
+// of the launch); longer (query, pair) work goes to the intra-task mode.
+constexpr int64_t CRIT_MIN_STEPS = 16384;
+constexpr double CRIT_FRACTION = 0.35;  // pairs longer than this are launched separately
 
 }  // namespace
 
@@ -91,6 +93,7 @@ struct sw_handle_s {
   DevBuf qcodes, qoff, matrix, prof, bbuf, bbuf_long, counters, ovf, ovf_count, scores_tmp, rbuf, qdesc;
   DevBuf glinks, gflags;  // superstrip boundary rows and their counters (long pairs)
   DevBuf rgrows, rflags;  // re-score: CTA-to-CTA rows, counters
+  DevBuf imap;            // short work item order
   int* pinned_count = nullptr;
   cudaEvent_t ev_begin = nullptr, ev_end = nullptr;
   bool search_timed = false;
@@ -98,8 +101,9 @@ struct sw_handle_s {
   std::vector<int> event_kind;
   // options
   int64_t opt_thr = 0, opt_G = 0, opt_R = 0;
-  int64_t opt_t_long = T_LONG;  // pairs longer than this use the intra-task (long) mode
+  int64_t opt_t_long = -1;      // >= 0: pairs longer than this always use the intra-task mode
   int64_t opt_query_pairs = 1;  // pair queries two per register for the short pairs
+  int64_t opt_pack_long = 0;    // 1: several long pairs per CTA item when a query has fewer strips than warps
   // last-search bookkeeping
   sw_stats_t stats{};
   cudaStream_t last_stream = nullptr;
@@ -232,6 +236,8 @@ int32_t sw_set_option(sw_handle_t h, const char* key, int64_t value) {
   } else if (k == "t_long") {
     if (value < 0) return set_err(h, SW_EINVAL, "t_long must be >= 0");
     h->opt_t_long = value;
+  } else if (k == "pack_long") {
+    h->opt_pack_long = value;
   } else if (k == "query_pairs") {
     h->opt_query_pairs = value;
   } else if (k == "timing_accumulate") {
@@ -261,7 +267,7 @@ int32_t sw_load_db(sw_handle_t h, const uint8_t* codes, const int64_t* offsets, 
     db->alpha = alphabet_size;
     Packed P;
     try {
-      pack_db(codes, offsets, n_seqs, alphabet_size, h->opt_t_long, P);
+      pack_db(codes, offsets, n_seqs, alphabet_size, h->opt_t_long >= 0 ? h->opt_t_long : T_LONG, P);
     } catch (const std::invalid_argument& e) {
       fail(SW_EINVAL, std::string("sw_load_db: ") + e.what());
     }
@@ -374,8 +380,7 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
   }
   std::vector<std::pair<int, int>> slot_m;
   for (auto& sl : slots) slot_m.push_back({ms[size_t(sl.k0)], sl.mode});
-  const int nlong_db = db->n_long;  // pairs longer than t_long
-  const int nshort_db = np - nlong_db;
+  const int nshort_db = np - db->n_long;  // (only for the geometry cost model)
   int G = 4, R = 24;
   choose_geom(h, slot_m, nshort_db > 0 ? db->sum_short_len / nshort_db : 1.0, G, R);
   if (!inter_config_supported(G, R)) fail(SW_EUNSUPPORTED, "no kernel for this geometry");
@@ -383,19 +388,40 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
   const int LB2 = (((R / 4) | 1) * 16);
   const int LS2 = G * LB2;
   const int SB2 = (((alpha + 1) * LS2 + 15) / 16) * 16;
-  // Per slot, pairs [0, nlong) go to the intra-task (long) mode: those longer
-  // than t_long, plus -- for very tall queries -- shorter pairs whose one-group
-  // critical path (strips x columns) would otherwise outlast the search.
+  // Per slot, pairs [0, nlong) go to the intra-task (long) mode: a short item
+  // (one lane group, every strip of its query in turn) must not run much longer
+  // than an average lane group's share of the whole launch, or it becomes the
+  // tail.  Optional override: "t_long" forces every pair longer than it there.
   auto pairs_longer_than = [&](int64_t Lc) {  // pairs are sorted longest first
     int lo = 0, hi = np;
     while (lo < hi) { const int mid = (lo + hi) / 2; if (db->pairs[size_t(mid)].len > Lc) lo = mid + 1; else hi = mid; }
     return lo;
   };
+  const int VG = G * (R % 8 == 0 ? 2 : 1);
+  double group_steps = 0;  // wavefront steps of all short work if nothing went long
+  for (auto& sl : slots) {
+    const int strips = std::max(1, (ms[size_t(sl.k0)] + G * R - 1) / (G * R));
+    const double seqs = sl.mode == 1 ? 2.0 * np : double(np);
+    const double cols = sl.mode == 1 ? 2.0 * db->len_prefix[size_t(np)] : double(db->len_prefix[size_t(np)]);
+    group_steps += double(strips) * (cols + seqs * VG);
+  }
+  const double resident_groups = 2.0 * h->sms * NG;
+  const double crit = std::max(double(CRIT_MIN_STEPS), CRIT_FRACTION * group_steps / resident_groups);
+  // Long-sequence databases (most residues in pairs longer than T_LONG, config 4)
+  // are scored entirely by the intra-task mode; otherwise the critical-path
+  // rule alone decides.
+  int nlong_opt = 0;
+  if (h->opt_t_long >= 0) {
+    nlong_opt = pairs_longer_than(h->opt_t_long);
+  } else {
+    const int nT = pairs_longer_than(T_LONG);
+    if (double(db->len_prefix[size_t(nT)]) > 0.5 * double(db->len_prefix[size_t(np)])) nlong_opt = nT;
+  }
   int nlong_max = 0;
   for (auto& sl : slots) {
     const int strips = std::max(1, (ms[size_t(sl.k0)] + G * R - 1) / (G * R));
-    const int64_t Lc = std::min<int64_t>(h->opt_t_long, CRIT_STEPS / strips);
-    sl.nlong = std::max(nlong_db, pairs_longer_than(Lc));
+    const int64_t Lc = int64_t(crit / strips);
+    sl.nlong = std::max(nlong_opt, pairs_longer_than(Lc));
     nlong_max = std::max(nlong_max, sl.nlong);
   }
   std::vector<int> qnlong(order.size(), 0);
@@ -450,12 +476,18 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
     // CTAs per long pair: enough to split very tall queries, few enough that each
     // CTA still runs ~LONG_ROUNDS rounds of W strips (amortises the pipeline ramp)
     d.n_super = std::max(1, (gl[k].n_strips + W * LONG_ROUNDS - 1) / (W * LONG_ROUNDS));
+    // a query with fewer strips than warps: several pairs per CTA item
+    d.pairs_per_item = (h->opt_pack_long && gl[k].n_strips < W) ? W / gl[k].n_strips : 1;
+    if (d.pairs_per_item > 1) d.n_super = 1;
+    d.pad2_ = 0;
     d.long_item_begin = int(long_items);
     d.flag_base = int(flags_total);
     d.done_base = int(done_total);
     d.glink_base = glink_total;
     d.glink_stride = db->lofs_host[size_t(nl)];
-    long_items += int64_t(nl) * d.n_super;
+    const int64_t items_q = d.pairs_per_item > 1 ? (nl + d.pairs_per_item - 1) / d.pairs_per_item
+                                                  : int64_t(nl) * d.n_super;
+    long_items += items_q;
     flags_total += int64_t(nl) * d.n_super;
     done_total += nl;
     if (d.n_super > 1) glink_total += int64_t(d.n_super) * d.glink_stride;
@@ -495,6 +527,36 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
       ++launches;
     }
   }
+  // global order of the short items: k-way merge of the slots' chunk lists
+  // (each already longest-first) by critical path = strips x first pair length
+  std::vector<int2> imap;
+  imap.reserve(size_t(item));
+  {
+    struct Head { double key; int slot, chunk; };
+    auto cmp = [](const Head& x, const Head& y) { return x.key < y.key || (x.key == y.key && x.slot > y.slot); };
+    std::vector<Head> heap;
+    auto key_of = [&](int j, int ch) {
+      const SlotDesc& d = sdesc[size_t(j)];
+      const int p = d.pair_begin + (d.mode == 1 ? (ch * NG) / 2 : ch * NG);
+      return double(d.n_strips) * double(db->pairs[size_t(std::min(p, np - 1))].len + 8);
+    };
+    for (size_t j = 0; j < sdesc.size(); ++j)
+      if (sdesc[j].n_items > 0) heap.push_back({key_of(int(j), 0), int(j), 0});
+    std::make_heap(heap.begin(), heap.end(), cmp);
+    while (!heap.empty()) {
+      std::pop_heap(heap.begin(), heap.end(), cmp);
+      Head hd = heap.back();
+      heap.pop_back();
+      imap.push_back(make_int2(hd.slot, hd.chunk));
+      if (hd.chunk + 1 < sdesc[size_t(hd.slot)].n_items) {
+        heap.push_back({key_of(hd.slot, hd.chunk + 1), hd.slot, hd.chunk + 1});
+        std::push_heap(heap.begin(), heap.end(), cmp);
+      }
+    }
+  }
+  SW_CK(h->imap.ensure(std::max<size_t>(imap.size(), 1) * sizeof(int2)));
+  if (!imap.empty())
+    SW_CK(cudaMemcpyAsync(h->imap.p, imap.data(), imap.size() * sizeof(int2), cudaMemcpyHostToDevice, c.st));
   SW_CK(h->qdesc.ensure(desc.size() * sizeof(QueryDesc) + sdesc.size() * sizeof(SlotDesc) + 16));
   QueryDesc* d_desc = h->qdesc.as<QueryDesc>();
   SlotDesc* d_slots = reinterpret_cast<SlotDesc*>(d_desc + desc.size());
@@ -527,6 +589,7 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
   a.slots = d_slots;
   a.n_slots = int(slots.size());
   a.n_short_items = item;
+  a.item_map = h->imap.as<int2>();
   a.SB2 = SB2;
   a.LS2 = LS2;
   a.LB2 = LB2;

@@ -348,6 +348,51 @@ __global__ void __launch_bounds__(NT) inter_kernel(InterArgs a) {
         if (a.queries[mid].long_item_begin <= item) lo = mid; else hi = mid - 1;
       }
       const QueryDesc d = a.queries[lo];
+      if (d.pairs_per_item > 1) {
+        // ---- query shorter than W strips: P = W / S pairs per CTA, S warps per
+        // pair (one strip each; upstream strips on higher warp ids)
+        const int S = d.n_strips_long, P = d.pairs_per_item;
+        const int grp = warp / S, jw = warp - grp * S;
+        const int pidx = (item - d.long_item_begin) * P + grp;
+        const bool active = grp < P && pidx < d.n_long;
+        uint32_t best = 0;
+        if (active) {
+          const PairRec pr = a.pairs[pidx];
+          const int s = S - 1 - jw;
+          uint8_t* myprof = lprof + warp * a.SBL;
+          {
+            const uint4* src = reinterpret_cast<const uint4*>(d.prof_long + (size_t)s * a.SBL);
+            uint4* dst = reinterpret_cast<uint4*>(myprof);
+            for (int i = lane; i < a.SBL / 16; i += 32) dst[i] = __ldg(src + i);
+          }
+          __syncwarp();
+          uint2* links = a.links + (size_t)blockIdx.x * W * a.lcap;
+          Link lk{};
+          const int wprod = warp + 1;  // the warp holding strip s-1 of this pair
+          lk.in = &s_prog[s > 0 ? wprod : warp];
+          lk.in_base = (s - 1) << 20;
+          lk.out = &s_prog[warp];
+          lk.out_base = s << 20;
+          strip_pass<32, LONG_R, true>(myprof, a.LSL, a.LBL, a.stream + pr.off, pr.len,
+                                       pr.len + 32 * SubLanes<LONG_R>::V, lane, s > 0, s + 1 < S,
+                                       links + (size_t)(s > 0 ? wprod : warp) * a.lcap,
+                                       links + (size_t)warp * a.lcap, lk, a.code_pad2, a.nGe, a.nGsGe, best);
+        }
+#pragma unroll
+        for (int o = 16; o > 0; o >>= 1) best = __vmaxs2(best, __shfl_xor_sync(FULL, best, o));
+        if (lane == 0) s_best[warp] = best;
+        __syncthreads();
+        if (tid < P) {
+          const int pj = (item - d.long_item_begin) * P + tid;
+          if (pj < d.n_long) {
+            uint32_t b = 0;
+            for (int w = tid * S; w < tid * S + S; ++w) b = __vmaxs2(b, s_best[w]);
+            emit_pair(a, d, pj, a.pairs[pj], b);
+          }
+        }
+        __syncthreads();
+        continue;
+      }
       const int K = d.n_super;               // CTAs sharing this pair
       const int64_t gstride = d.glink_stride;
       const int local = item - d.long_item_begin;
@@ -434,16 +479,12 @@ __global__ void __launch_bounds__(NT) inter_kernel(InterArgs a) {
         }
       }
     } else {
-      // ---------------- short work: find the slot of this item (slots are few)
-      const int c = item - n_long_items;
-      int lo = 0, hi = a.n_slots - 1;
-      while (lo < hi) {
-        const int mid = (lo + hi + 1) >> 1;
-        if (a.slots[mid].item_begin <= c) lo = mid; else hi = mid - 1;
-      }
-      const int sl = lo;
+      // ---------------- short work: the host ordered all (slot, chunk) items of
+      // the launch by critical path (strips x pair length), longest first
+      const int2 sc = a.item_map[item - n_long_items];
+      const int sl = sc.x;
       const SlotDesc d = a.slots[sl];
-      const int chunk = c - d.item_begin;
+      const int chunk = sc.y;
       const bool q2 = d.mode == 1;
       int p, half = 0;
       if (q2) {  // chunk of NG half-pairs: DB sequence = one half of a pair

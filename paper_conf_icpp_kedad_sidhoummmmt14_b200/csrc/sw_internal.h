@@ -63,6 +63,8 @@ struct QueryDesc {
   int flag_base;             // this query's superstrip counters: gflags[flag_base + pair * n_super + k]
   int done_base;             // per-pair superstrip completion counters: gdone[done_base + pair]
   int n_long;                // pairs [0, n_long) are this query's long items
+  int pairs_per_item;        // > 1: the query has fewer than W strips; a long item holds W/strips pairs
+  int pad2_;
   int64_t glink_base;        // boundary rows: glinks[glink_base + c * glink_stride + lofs[pair] ...]
   int64_t glink_stride;      // sum over this query's long pairs of (len + 72)
 };
@@ -89,6 +91,7 @@ struct InterArgs {
   const SlotDesc* slots;     // [n_slots] short-pair work
   int n_slots;
   int n_short_items;         // sum of slots' n_items
+  const int2* item_map;      // short item -> (slot, chunk), longest critical path first
   int SB, LS, LB;            // short geometry (G, R of the launch), mode 0 profile
   int SB2, LS2, LB2;         // mode 1 (query-pair) profile
   int SBL, LSL, LBL;         // long geometry (32 lanes x LONG_R rows)

@@ -82,6 +82,36 @@ __global__ void k_cell(uint32_t* out, uint32_t seed) {
   if (best == 0x12345678u) out[blockIdx.x] = best;
 }
 
+// Same, with the production formulation: D = Hdiag + S on the FMA pipe,
+// H = max3(D, E, F), running max over D -> 3.5 ALU ops per cell pair.
+template <int R, bool PERM>
+__global__ void k_cell2(uint32_t* out, uint32_t seed) {
+  uint32_t H[R], E[R], S[R];
+  const uint32_t nge = 0xfffefffeu, ngsge = 0xfff4fff4u;
+#pragma unroll
+  for (int r = 0; r < R; ++r) { H[r] = (seed + r) & 0x00ff00ffu; E[r] = 0; S[r] = ((r * 3 + threadIdx.x) & 7) * 0x00010001u; }
+  uint32_t best = 0, hdiag = 0;
+  for (int it = 0; it < ITERS / 4; ++it) {
+    uint32_t F = 0, hd = hdiag, dprev = 0;
+#pragma unroll
+    for (int r = 0; r < R; ++r) {
+      const uint32_t dg = __vadd2(hd, S[r]);
+      const uint32_t h = __vimax3_s16x2(dg, E[r], F);
+      const uint32_t t = __vadd2(h, ngsge);
+      E[r] = __viaddmax_s16x2_relu(E[r], nge, t);
+      F = __viaddmax_s16x2_relu(F, nge, t);
+      hd = H[r]; H[r] = h;
+      if (r & 1) best = __vimax3_s16x2(best, dprev, dg); else dprev = dg;
+    }
+    hdiag = F ^ it;
+    if constexpr (PERM) {
+#pragma unroll
+      for (int r = 0; r < R; ++r) S[r] = __byte_perm(S[r], S[(r + 1) % R], 0x5432);
+    }
+  }
+  if (best == 0x12345678u) out[blockIdx.x] = best;
+}
+
 __global__ void k_clock(unsigned long long* t) {
   unsigned long long c0 = clock64();
   uint32_t x = threadIdx.x;
@@ -147,6 +177,11 @@ int main() {
     mc = time_kernel(k_cell<32, false>, sms * g, block, d_out);
     cells = double(sms * g) * block * (ITERS / 4) * 32 * 2;
     printf("{\"probe\":\"gotoh_cellpair_R32_noperm\",\"blocks_per_sm\":%d,\"ms\":%.4f,\"GCUPS\":%.1f}\n", g, mc, cells / (mc * 1e6));
+  }
+  for (int g = 1; g <= 4; g *= 2) {
+    float mc = time_kernel(k_cell2<24, false>, sms * g, block, d_out);
+    double cells = double(sms * g) * block * (ITERS / 4) * 24 * 2;
+    printf("{\"probe\":\"gotoh_cellpair_D_max3_R24\",\"blocks_per_sm\":%d,\"ms\":%.4f,\"GCUPS\":%.1f}\n", g, mc, cells / (mc * 1e6));
   }
   CK(cudaGetLastError());
   return 0;

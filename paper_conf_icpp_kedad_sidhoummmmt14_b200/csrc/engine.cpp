@@ -749,8 +749,11 @@ int32_t sw_search(sw_handle_t h, const uint8_t* q_codes, const int64_t* q_offset
         for (auto L : qlen) mmax = std::max(mmax, L);
         const int rows_per_strip = 32 * RESCORE_R;
         const int nstrips = int((mmax + rows_per_strip - 1) / rows_per_strip);
-        const int K = std::max(1, (nstrips + RESCORE_WARPS * LONG_ROUNDS - 1) / (RESCORE_WARPS * LONG_ROUNDS));
-        const int grid = std::max(1, std::min<int>(cnt * K, h->sms * 2));
+        // one strip per warp (a single round): CTA c only waits on CTA c-1,
+        // which took its item earlier, so any grid size is deadlock-free and
+        // the pair's critical path is its columns + strips x (32 + lag)
+        const int K = std::max(1, (nstrips + RESCORE_WARPS - 1) / RESCORE_WARPS);
+        const int grid = std::max(1, std::min<int>(cnt * K, h->sms * 4));
         const int bcap = Lmax + 32 + 72;
         SW_CK(h->rbuf.ensure(size_t(grid) * RESCORE_WARPS * bcap * sizeof(int2)));
         SW_CK(h->rgrows.ensure(size_t(cnt) * K * bcap * sizeof(int2) + 16));

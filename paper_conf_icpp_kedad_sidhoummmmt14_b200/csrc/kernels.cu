@@ -28,6 +28,7 @@ constexpr int8_t PAD_SCORE = -64;  // S[.][PAD] = S[PAD][.] <= 0 (reading R-12)
 // producer is this many columns ahead, so producer and consumer warps of a
 // chain run decoupled instead of in lock-step (the consumer then rarely waits).
 constexpr int LINK_LAG = 64;
+constexpr int RESCORE_LAG = 16;  // re-score chains: one round per CTA, short lag keeps the critical path short
 
 // ---------------------------------------------------------------------------
 // Query profile: prof[s][a][k][r] = S[q[s*G*R + k*R + r]][a]  (int8)
@@ -682,7 +683,7 @@ __global__ void __launch_bounds__(RESCORE_WARPS * 32) rescore_kernel(RescoreArgs
       uint2 cw = make_uint2(padw, padw);
       int2 tb0 = z2, tb1 = z2, tb2 = z2, tb3 = z2;
       int seen = -1;
-      if (rd && L > 0) wait_progress(lk, lk.in_base + min(4 + 31 + LINK_LAG, L + 32), seen);
+      if (rd && L > 0) wait_progress(lk, lk.in_base + min(4 + 31 + RESCORE_LAG, L + 32), seen);
       if (lead && L > 0) {
         cw = codes[0];
         if (rd) { tb0 = __ldcg(rp + 0); tb1 = __ldcg(rp + 1); tb2 = __ldcg(rp + 2); tb3 = __ldcg(rp + 3); }
@@ -691,7 +692,7 @@ __global__ void __launch_bounds__(RESCORE_WARPS * 32) rescore_kernel(RescoreArgs
       for (int t0 = 0; t0 < T; t0 += 4) {
         const uint2 cwc = cw;
         const int2 c0 = tb0, c1 = tb1, c2 = tb2, c3 = tb3;
-        if (rd && t0 + 4 < L) wait_progress(lk, lk.in_base + min(t0 + 8 + 31 + LINK_LAG, L + 32), seen);
+        if (rd && t0 + 4 < L) wait_progress(lk, lk.in_base + min(t0 + 8 + 31 + RESCORE_LAG, L + 32), seen);
         if (lead) {
           if (t0 + 4 < L) {
             cw = codes[(t0 + 4) >> 2];

@@ -150,7 +150,7 @@ cudaError_t launch_inter(int G, int R, int NT, int grid, int smem_bytes, const I
 bool inter_config_supported(int G, int R);
 int inter_block_threads();  // NT of the scoring kernel (its long items use NT/32 chained warps)
 cudaError_t launch_rescore(int grid, const RescoreArgs& a, cudaStream_t st);
-constexpr int RESCORE_WARPS = 16;
+constexpr int RESCORE_WARPS = 8;
 constexpr int RESCORE_R = 8;
 
 }  // namespace swdual

@@ -108,8 +108,9 @@ typedef struct {
   double cells;            /* sum_q m_q * sum_d n_d of the last search (real residues)      */
   double cells_short;      /* of which in pairs of length <= 3000 (the bulk launches)        */
   double cells_computed;   /* cell updates issued incl. row/column padding and wave fill     */
-  double short_ms;         /* summed CUDA-event time of the short-pair scoring launches      */
-  double long_ms;          /* summed CUDA-event time of the long-pair launches (overlapped)  */
+  double short_ms;         /* summed CUDA-event time of the scoring launches (the persistent  */
+                           /* kernel covers long AND short pairs of the search)             */
+  double long_ms;          /* reserved (0): long pairs run inside the same persistent launch */
   double search_ms;        /* device time of the whole search, first upload to last kernel   */
   int32_t n_launches;      /* kernels launched by the last search                           */
   int32_t n_score_launches;/* of which scoring (inter-task) kernels                         */

@@ -103,6 +103,7 @@ struct sw_handle_s {
   int64_t opt_thr = 0, opt_G = 0, opt_R = 0;
   int64_t opt_t_long = -1;      // >= 0: pairs longer than this always use the intra-task mode
   int64_t opt_query_pairs = 1;  // pair queries two per register for the short pairs
+  int64_t opt_bank_copy = 1;    // query-pair profile: second smem copy shifted by 64 B for odd lane groups
   int64_t opt_pack_long = 0;    // 1: several long pairs per CTA item when a query has fewer strips than warps
   // last-search bookkeeping
   sw_stats_t stats{};
@@ -152,12 +153,18 @@ static int32_t guarded(sw_handle_s* h, F&& f) {
 // ----------------------------------------------------------------------------
 // geometry of the inter-task kernel for a query of m rows and a launch whose
 // pairs average Lavg columns
-static ProfGeom make_geom(int G, int R, int m, int alpha, bool dense = false) {
+// long = true: the intra-task (G = 32) unit-interleaved layout, LB = the unit
+// (8 bytes, the lane's offset); otherwise lane blocks of an odd number of units,
+// letters padded to a multiple of 128 B when bank-spread copies are used.
+static ProfGeom make_geom(int G, int R, int m, int alpha, bool long_mode = false, bool pad128 = false) {
   ProfGeom g{};
   g.G = G;
   g.R = R;
-  g.LB = dense ? R : ((R % 8 == 0) ? (((R / 8) | 1) * 8) : (((R / 4) | 1) * 4));
-  g.LS = G * g.LB;
+  g.UB = (R % 8 == 0) ? 8 : 4;
+  g.il = (long_mode && SW_LONG_IL) ? 1 : 0;
+  g.LB = long_mode ? (SW_LONG_IL ? g.UB : R) : ((R % 8 == 0) ? (((R / 8) | 1) * 8) : (((R / 4) | 1) * 4));
+  g.LS = long_mode ? G * R : G * g.LB;
+  if (pad128) g.LS = ((g.LS + 127) / 128) * 128;
   g.NL = alpha + 1;
   g.SB = ((g.NL * g.LS + 15) / 16) * 16;
   g.n_strips = std::max(1, (m + G * R - 1) / (G * R));
@@ -238,6 +245,8 @@ int32_t sw_set_option(sw_handle_t h, const char* key, int64_t value) {
     h->opt_t_long = value;
   } else if (k == "pack_long") {
     h->opt_pack_long = value;
+  } else if (k == "bank_copy") {
+    h->opt_bank_copy = value;
   } else if (k == "query_pairs") {
     h->opt_query_pairs = value;
   } else if (k == "timing_accumulate") {
@@ -386,8 +395,17 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
   if (!inter_config_supported(G, R)) fail(SW_EUNSUPPORTED, "no kernel for this geometry");
   const int NT = inter_block_threads(), NG = NT / G, W = NT / 32;
   const int LB2 = (((R / 4) | 1) * 16);
-  const int LS2 = G * LB2;
+  // Query-pair profile rows are LDS.128 per lane: a quarter-warp phase holds two
+  // G = 4 groups reading random letters.  With LS2 a multiple of 128 B and odd
+  // groups reading a second copy shifted by 64 B, the two groups always hit
+  // disjoint bank halves ({k*LB2} mod 128 and {k*LB2 + 64} mod 128 partition
+  // the eight 16-byte slots when LB2 is an odd multiple of 16).
+  const bool bank_copy = h->opt_bank_copy != 0;
+  const int LS2 = bank_copy ? ((G * LB2 + 127) / 128) * 128 : G * LB2;
   const int SB2 = (((alpha + 1) * LS2 + 15) / 16) * 16;
+  // copies: lanes of one phase (128 B / unit) divided by the group width
+  const int ncopy2 = bank_copy ? std::max(1, (128 / 16) / G) : 1;
+  const int ncopy0 = bank_copy ? std::max(1, (128 / (R % 8 == 0 ? 8 : 4)) / G) : 1;
   // Per slot, pairs [0, nlong) go to the intra-task (long) mode: a short item
   // (one lane group, every strip of its query in turn) must not run much longer
   // than an average lane group's share of the whole launch, or it becomes the
@@ -434,11 +452,11 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
   std::vector<ProfGeom> gl;
   std::vector<size_t> off_l;
   for (size_t k = 0; k < order.size(); ++k) {
-    gl.push_back(make_geom(32, LONG_R, ms[k], alpha, /*dense=*/true));
+    gl.push_back(make_geom(32, LONG_R, ms[k], alpha, /*long_mode=*/true));
     off_l.push_back(total);
     total += qnlong[k] > 0 ? size_t(gl.back().n_strips) * gl.back().SB : 0;
   }
-  const ProfGeom g1 = make_geom(G, R, 1, alpha);  // SB / LS / LB of the mode-0 profile
+  const ProfGeom g1 = make_geom(G, R, 1, alpha, false, bank_copy);  // SB / LS / LB of the mode-0 profile
   std::vector<size_t> off_s;
   std::vector<int> strips_s;
   for (auto& sl : slots) {
@@ -516,7 +534,7 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
       const double sumS = pair_len_sum(sl.nlong, np) + double(ns) * 2 * G;
       if (sl.mode == 1) {
         SW_CK(launch_build_profile_q2(qptr(sl.k0), ms[size_t(sl.k0)], qptr(sl.k1), ms[size_t(sl.k1)], dmat, alpha,
-                                      G, R, LB2, d.n_strips, SB2, prof + off_s[j], c.st));
+                                      G, R, LB2, LS2, d.n_strips, SB2, prof + off_s[j], c.st));
         cells_computed += 2.0 * (2.0 * sumS) * double(d.n_strips) * G * R;  // every sequence, 2 queries
       } else {
         ProfGeom gq = g1;
@@ -565,7 +583,14 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
   int max_strips = 1;
   for (int n : strips_s) max_strips = std::max(max_strips, n);
   const ProfGeom l0 = gl[0];
-  const int smem = std::max(g1.SB, SB2) + (nlong_max > 0 ? W * l0.SB : 0);
+  // copy c of a strip sits at c * cstride; cstride = SB + 128 / ncopy (SB is a
+  // multiple of 128 when copies are used)
+  const int cstride0 = g1.SB + (ncopy0 > 1 ? 128 / ncopy0 : 0);
+  const int cstride2 = SB2 + (ncopy2 > 1 ? 128 / ncopy2 : 0);
+  const int sprof_bytes = std::max((ncopy0 - 1) * cstride0 + g1.SB, (ncopy2 - 1) * cstride2 + SB2);
+  // an item is either short or long: the long-mode slots reuse the same bytes
+  const int smem = SW_SMEM_UNION ? std::max(sprof_bytes, nlong_max > 0 ? W * l0.SB : 0)
+                                 : sprof_bytes + (nlong_max > 0 ? W * l0.SB : 0);
   const int occ = inter_max_ctas_per_sm(G, R, NT, smem);
   if (occ <= 0) fail(SW_ECUDA, "inter kernel does not fit on an SM");
   const int64_t n_items = long_items + item;
@@ -591,6 +616,10 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
   a.n_short_items = item;
   a.item_map = h->imap.as<int2>();
   a.SB2 = SB2;
+  a.ncopy[0] = ncopy0;
+  a.ncopy[1] = ncopy2;
+  a.cstride[0] = cstride0;
+  a.cstride[1] = cstride2;
   a.LS2 = LS2;
   a.LB2 = LB2;
   a.SB = g1.SB;

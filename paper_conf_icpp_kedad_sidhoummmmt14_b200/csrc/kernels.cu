@@ -44,9 +44,17 @@ __global__ void build_profile_kernel(const uint8_t* __restrict__ q, int m, const
     if (rem < g.NL * g.LS) {
       const int a = rem / g.LS;
       const int rr = rem - a * g.LS;
-      const int k = rr / g.LB;
-      const int r = rr - k * g.LB;
-      if (r < g.R) {
+      int k, r;
+      if (g.il) {  // [unit u][lane k][UB bytes]
+        const int u = rr / (g.G * g.UB);
+        const int w = rr - u * (g.G * g.UB);
+        k = w / g.UB;
+        r = u * g.UB + (w - k * g.UB);
+      } else {     // [lane k][LB bytes] (LS may be padded past G lanes)
+        k = rr / g.LB;
+        r = rr - k * g.LB;
+      }
+      if (k < g.G && r < g.R) {
         const int row = s * g.G * g.R + k * g.R + r;
         v = (row < m && a < alpha) ? M[q[row] * alpha + a] : PAD_SCORE;
       }
@@ -69,8 +77,7 @@ cudaError_t launch_build_profile(const uint8_t* q, int m, const int8_t* matrix, 
 //   low 16 = S[qa[row]][a], high 16 = S[qb[row]][a]  (PAD rows / letters: PAD_SCORE)
 __global__ void build_profile_q2_kernel(const uint8_t* __restrict__ qa, int ma, const uint8_t* __restrict__ qb,
                                         int mb, const int8_t* __restrict__ M, int alpha, int G, int R, int LB2,
-                                        int n_strips, int SB2, uint32_t* __restrict__ prof) {
-  const int LS2 = G * LB2;
+                                        int LS2, int n_strips, int SB2, uint32_t* __restrict__ prof) {
   const int64_t total = (int64_t)n_strips * (SB2 / 4);
   for (int64_t i = blockIdx.x * (int64_t)blockDim.x + threadIdx.x; i < total;
        i += (int64_t)gridDim.x * blockDim.x) {
@@ -82,7 +89,7 @@ __global__ void build_profile_q2_kernel(const uint8_t* __restrict__ qa, int ma, 
       const int rr = rem - a * LS2;
       const int k = rr / LB2;
       const int r = (rr - k * LB2) / 4;
-      if (r < R) {
+      if (k < G && r < R) {
         const int row = s * G * R + k * R + r;
         const int va = (row < ma && a < alpha) ? M[qa[row] * alpha + a] : PAD_SCORE;
         const int vb = (row < mb && a < alpha) ? M[qb[row] * alpha + a] : PAD_SCORE;
@@ -94,13 +101,13 @@ __global__ void build_profile_q2_kernel(const uint8_t* __restrict__ qa, int ma, 
 }
 
 cudaError_t launch_build_profile_q2(const uint8_t* qa, int ma, const uint8_t* qb, int mb, const int8_t* matrix,
-                                    int alpha, int G, int R, int LB2, int n_strips, int SB2, uint8_t* prof,
+                                    int alpha, int G, int R, int LB2, int LS2, int n_strips, int SB2, uint8_t* prof,
                                     cudaStream_t st) {
   const int64_t total = (int64_t)n_strips * (SB2 / 4);
   int grid = int((total + 255) / 256);
   if (grid > 4096) grid = 4096;
   if (grid < 1) grid = 1;
-  build_profile_q2_kernel<<<grid, 256, 0, st>>>(qa, ma, qb, mb, matrix, alpha, G, R, LB2, n_strips, SB2,
+  build_profile_q2_kernel<<<grid, 256, 0, st>>>(qa, ma, qb, mb, matrix, alpha, G, R, LB2, LS2, n_strips, SB2,
                                                 reinterpret_cast<uint32_t*>(prof));
   return cudaGetLastError();
 }
@@ -174,7 +181,7 @@ struct SubLanes {
   static constexpr int V = (R % 8 == 0) ? 2 : 1;
 };
 
-template <int G, int R, bool LINKED, bool Q2 = false>
+template <int G, int R, bool LINKED, bool Q2 = false, int US = (Q2 ? 16 : ((R % 8 == 0) ? 8 : 4))>
 __device__ __forceinline__ void strip_pass(const uint8_t* sprof, int LS, int LB, const uint16_t* pstream, int L,
                                            int T, int k, bool rd, bool wr, const uint2* __restrict__ rp,
                                            uint2* __restrict__ wp, const Link& lk, uint32_t code_pad2,
@@ -182,9 +189,9 @@ __device__ __forceinline__ void strip_pass(const uint8_t* sprof, int LS, int LB,
   constexpr int V = SubLanes<R>::V;
   constexpr int VG = V * G;   // width of the wave in sub-lanes
   constexpr int RH = R / V;   // rows per sub-lane
-  uint32_t HA[R], HB[R], E[R];
+  uint32_t HA[R], E[R];
 #pragma unroll
-  for (int r = 0; r < R; ++r) { HA[r] = 0; HB[r] = 0; E[r] = 0; }
+  for (int r = 0; r < R; ++r) { HA[r] = 0; E[r] = 0; }
   uint32_t hdiag = 0, sH = 0, sF = 0, sC = code_pad2;
   const uint2* __restrict__ codes = reinterpret_cast<const uint2*>(pstream);
   const uint32_t pad4 = code_pad2 | (code_pad2 << 16);
@@ -193,8 +200,9 @@ __device__ __forceinline__ void strip_pass(const uint8_t* sprof, int LS, int LB,
   const uint2 z2 = make_uint2(0, 0);
   // second sub-lane: its inputs are the first sub-lane's outputs of the previous step
   uint32_t hdiag1 = 0, cH = 0, cF = 0, pC = code_pad2;
-  const uint8_t* pad_row = sprof + (code_pad2 & 0xffu) * LS + laneoff;
-  const uint8_t *ppa = pad_row, *ppb = pad_row;
+  const uint32_t sbase = static_cast<uint32_t>(__cvta_generic_to_shared(sprof));
+  const uint32_t pad_row = sbase + (code_pad2 & 0xffu) * LS + laneoff;
+  uint32_t ppa = pad_row, ppb = pad_row;
   rp += VG - 1;  // sub-lane 0 of lane 0 reads column c at rp[c + VG - 1]
 
   // lane 0 prefetch of block 0: 4 columns of codes and (if rd) 4 boundary cells.
@@ -241,25 +249,19 @@ __device__ __forceinline__ void strip_pass(const uint8_t* sprof, int LS, int LB,
         rH = tv.x;
         rF = tv.y;
       }
-      const uint8_t* pa;
-      const uint8_t* pb;
+      uint32_t pa, pb;
       if constexpr (Q2) {  // one DB sequence (byte `shift` of the pair word) against two queries
-        pa = sprof + ((rC >> shift) & 0xffu) * LS + laneoff;
+        pa = sbase + ((rC >> shift) & 0xffu) * LS + laneoff;
         pb = pa;
       } else {
-        pa = sprof + (rC & 0xffu) * LS + laneoff;
-        pb = sprof + (rC >> 8) * LS + laneoff;
+        pa = sbase + (rC & 0xffu) * LS + laneoff;
+        pb = sbase + (rC >> 8) * LS + laneoff;
       }
-      // even steps read HA and write HB, odd steps the reverse (4 steps per block)
       if constexpr (V == 2) {
         uint32_t h1 = cH, f1 = cF;
-        if (j & 1) {
-          gotoh_rows<R, RH, R, Q2>(HB, HA, E, best, hdiag1, ppa, ppb, h1, f1, nGe, nGsGe);
-          gotoh_rows<R, 0, RH, Q2>(HB, HA, E, best, hdiag, pa, pb, rH, rF, nGe, nGsGe);
-        } else {
-          gotoh_rows<R, RH, R, Q2>(HA, HB, E, best, hdiag1, ppa, ppb, h1, f1, nGe, nGsGe);
-          gotoh_rows<R, 0, RH, Q2>(HA, HB, E, best, hdiag, pa, pb, rH, rF, nGe, nGsGe);
-        }
+        // sub-lane 1 (rows RH..R-1, column t-1) first: it reads rows it owns only
+        gotoh_rows_inplace<R, RH, R, Q2, US>(HA, E, best, hdiag1, ppa, ppb, h1, f1, nGe, nGsGe);
+        gotoh_rows_inplace<R, 0, RH, Q2, US>(HA, E, best, hdiag, pa, pb, rH, rF, nGe, nGsGe);
         cH = rH;
         cF = rF;
         ppa = pa;
@@ -269,8 +271,7 @@ __device__ __forceinline__ void strip_pass(const uint8_t* sprof, int LS, int LB,
         sC = pC;
         pC = rC;
       } else {
-        if (j & 1) gotoh_rows<R, 0, R, Q2>(HB, HA, E, best, hdiag, pa, pb, rH, rF, nGe, nGsGe);
-        else gotoh_rows<R, 0, R, Q2>(HA, HB, E, best, hdiag, pa, pb, rH, rF, nGe, nGsGe);
+        gotoh_rows_inplace<R, 0, R, Q2, US>(HA, E, best, hdiag, pa, pb, rH, rF, nGe, nGsGe);
         sH = rH;
         sF = rF;
         sC = rC;
@@ -318,8 +319,10 @@ __device__ __forceinline__ void emit_pair(const InterArgs& a, const QueryDesc& d
 template <int G, int R, int NT>
 __global__ void __launch_bounds__(NT) inter_kernel(InterArgs a) {
   extern __shared__ __align__(16) uint8_t smem[];
-  uint8_t* sprof = smem;                         // short-mode strip profile (max(SB, SB2) bytes)
-  uint8_t* lprof = smem + max(a.SB, a.SB2);      // long mode: one a.SBL slot per warp
+  // An item is either short or long, so the two uses share shared memory:
+  uint8_t* sprof = smem;                         // short mode: the strip profile (bank-spread copies)
+  uint8_t* lprof = smem + (SW_SMEM_UNION ? 0 : max(a.cstride[0] * (a.ncopy[0] - 1) + a.SB,
+                                                    a.cstride[1] * (a.ncopy[1] - 1) + a.SB2));  // long mode: one a.SBL slot per warp
   __shared__ int s_item;
   __shared__ int s_prog[NT / 32];
   __shared__ uint32_t s_best[NT / 32];
@@ -341,6 +344,7 @@ __global__ void __launch_bounds__(NT) inter_kernel(InterArgs a) {
     const int item = s_item;
     if (item >= n_items) break;
     if (item < n_long_items) {
+      loaded = -1;  // the long-mode slots overwrite the short strip profile
       // ---------------- long pair, superstrip k: W chained strips on this CTA's
       // warps; superstrips k-1 / k+1 of the same pair run on other CTAs
       int lo = 0, hi = a.n_queries - 1;
@@ -374,7 +378,7 @@ __global__ void __launch_bounds__(NT) inter_kernel(InterArgs a) {
           lk.in_base = (s - 1) << 20;
           lk.out = &s_prog[warp];
           lk.out_base = s << 20;
-          strip_pass<32, LONG_R, true>(myprof, a.LSL, a.LBL, a.stream + pr.off, pr.len,
+          strip_pass<32, LONG_R, true, false, LONG_US>(myprof, a.LSL, a.LBL, a.stream + pr.off, pr.len,
                                        pr.len + 32 * SubLanes<LONG_R>::V, lane, s > 0, s + 1 < S,
                                        links + (size_t)(s > 0 ? wprod : warp) * a.lcap,
                                        links + (size_t)warp * a.lcap, lk, a.code_pad2, a.nGe, a.nGsGe, best);
@@ -448,7 +452,7 @@ __global__ void __launch_bounds__(NT) inter_kernel(InterArgs a) {
           lk.out_gpu = true;
         }
         lk.out_base = s << 20;
-        strip_pass<32, LONG_R, true>(myprof, a.LSL, a.LBL, a.stream + pr.off, pr.len, T, lane, rd, wr, rp, wp, lk,
+        strip_pass<32, LONG_R, true, false, LONG_US>(myprof, a.LSL, a.LBL, a.stream + pr.off, pr.len, T, lane, rd, wr, rp, wp, lk,
                                      a.code_pad2, a.nGe, a.nGsGe, best);
       }
 #pragma unroll
@@ -504,20 +508,22 @@ __global__ void __launch_bounds__(NT) inter_kernel(InterArgs a) {
       if (G < 32) T = __reduce_max_sync(FULL, T);  // warp-uniform trip count (shuffles)
       uint32_t best = 0;
       const int SBx = q2 ? a.SB2 : a.SB;
+      const int ncp = q2 ? a.ncopy[1] : a.ncopy[0], csx = q2 ? a.cstride[1] : a.cstride[0];
+      const uint8_t* gprof = sprof + (g & (ncp - 1)) * csx;  // this group's bank-spread copy
       for (int s = 0; s < d.n_strips; ++s) {
         const int want = (sl << 16) | s;
         if (want != loaded) {
           __syncthreads();
-          copy_strip(sprof, d.prof + (size_t)s * SBx, SBx);
+          for (int cp = 0; cp < ncp; ++cp) copy_strip(sprof + cp * csx, d.prof + (size_t)s * SBx, SBx);
           __syncthreads();
           loaded = want;
         }
         if (q2)
-          strip_pass<G, R, false, true>(sprof, a.LS2, a.LB2, a.stream + pr.off, pr.len, T, k, s > 0,
+          strip_pass<G, R, false, true>(gprof, a.LS2, a.LB2, a.stream + pr.off, pr.len, T, k, s > 0,
                                         s + 1 < d.n_strips, bb, bb, Link{}, a.code_pad2,
                                         a.nGe, a.nGsGe, best, half ? 8u : 0u);
         else
-          strip_pass<G, R, false>(sprof, a.LS, a.LB, a.stream + pr.off, pr.len, T, k, s > 0, s + 1 < d.n_strips,
+          strip_pass<G, R, false>(gprof, a.LS, a.LB, a.stream + pr.off, pr.len, T, k, s > 0, s + 1 < d.n_strips,
                                   bb, bb, Link{}, a.code_pad2, a.nGe, a.nGsGe, best);
       }
 #pragma unroll

@@ -44,65 +44,89 @@ __host__ __device__ constexpr int lane_block_bytes(int R) {
   return ((R % 8 == 0) ? (((R / 8) | 1) * 8) : (((R / 4) | 1) * 4));
 }
 
+// Shared-memory loads by 32-bit shared-window address (the profile pointers
+// stay 32-bit: fewer registers than generic 64-bit pointers, no address
+// rematerialisation in the hot loop).
+__device__ __forceinline__ uint4 lds128(uint32_t a) {
+  uint4 v;
+  asm volatile("ld.shared.v4.u32 {%0, %1, %2, %3}, [%4];" : "=r"(v.x), "=r"(v.y), "=r"(v.z), "=r"(v.w) : "r"(a));
+  return v;
+}
+__device__ __forceinline__ uint2 lds64(uint32_t a) {
+  uint2 v;
+  asm volatile("ld.shared.v2.u32 {%0, %1}, [%2];" : "=r"(v.x), "=r"(v.y) : "r"(a));
+  return v;
+}
+__device__ __forceinline__ uint32_t lds32(uint32_t a) {
+  uint32_t v;
+  asm volatile("ld.shared.u32 %0, [%1];" : "=r"(v) : "r"(a));
+  return v;
+}
+
 // Rows [R0, R1) of one column for one lane (a "sub-lane"; R0 = 0, R1 = R is
-// the whole lane).
-//   Hin[r] : H_{r,j-1} (previous column);  Hout[r] : out H_{r,j}  (the caller
-//            alternates two buffers, so the diagonal needs no register moves)
+// the whole lane), ONE H buffer updated in place: the diagonal term of row r+1,
+// D_{r+1} = H_{r,j-1} + S, is formed BEFORE H[r] is overwritten with H_{r,j},
+// so the old value dies as the new one is born and H[r] keeps one register
+// across columns (no second buffer, no moves).
+//   H[r]   : in H_{r,j-1}, out H_{r,j}
 //   E[r]   : in E_{r,j},   out E_{r,j+1}
 //   hdiag  : in H_{R0-1, j-1}, out H_{R0-1, j}  (top boundary of the previous column)
 //   Hio    : in H_{R0-1, j} (from above), out H_{R1-1, j}
 //   Fio    : in F_{R0, j},                out F_{R1, j}
-// Q2 = false: pa / pb point at the int8 profile rows of the two DB letters of a
-//   pair (one per s16x2 half), combined per row by a sign-extending PRMT.
-// Q2 = true:  pa points at s16x2 profile words (two queries, one DB letter).
-template <int R, int R0, int R1, bool Q2>
-__device__ __forceinline__ void gotoh_rows(const uint32_t (&Hin)[R], uint32_t (&Hout)[R], uint32_t (&E)[R],
-                                           uint32_t& best, uint32_t& hdiag, const uint8_t* __restrict__ pa,
-                                           const uint8_t* __restrict__ pb, uint32_t& Hio, uint32_t& Fio,
-                                           uint32_t nGe, uint32_t nGsGe) {
+// Q2 = false: pa / pb are the shared addresses of the int8 profile rows of the
+//   two DB letters of a pair (one per s16x2 half), combined per row by a
+//   sign-extending PRMT.
+// Q2 = true:  pa addresses s16x2 profile words (two queries, one DB letter).
+// US: bytes between consecutive load units of one lane (= the unit size for the
+// lane-blocked layout; G * unit for the unit-interleaved long-mode layout).
+template <int R, int R0, int R1, bool Q2, int US = (Q2 ? 16 : ((R % 8 == 0) ? 8 : 4))>
+__device__ __forceinline__ void gotoh_rows_inplace(uint32_t (&H)[R], uint32_t (&E)[R], uint32_t& best,
+                                                   uint32_t& hdiag, uint32_t pa, uint32_t pb, uint32_t& Hio,
+                                                   uint32_t& Fio,
+                                                   uint32_t nGe, uint32_t nGsGe) {
   static_assert(R0 % 4 == 0 && (R1 - R0) % 4 == 0 && R1 <= R, "row range must be 4-aligned");
-  uint32_t hd = hdiag;
-  hdiag = Hio;
-  uint32_t F = Fio;
-  uint32_t dprev = 0;
-  constexpr int UB = Q2 ? 4 : ((R % 8 == 0 && R0 % 8 == 0 && (R1 - R0) % 8 == 0) ? 8 : 4);  // rows per load
+  constexpr int N = R1 - R0;
+  uint32_t sv[N];  // S(q_r, letter) for the rows of this sub-lane
+  constexpr int UB = Q2 ? 4 : ((R % 8 == 0 && R0 % 8 == 0 && N % 8 == 0) ? 8 : 4);
 #pragma unroll
   for (int u = R0 / UB; u < R1 / UB; ++u) {
-    uint32_t sv[UB];
+    const int b = u * UB - R0;
     if constexpr (Q2) {
-      const uint4 w = *reinterpret_cast<const uint4*>(pa + u * 16);
-      sv[0] = w.x; sv[1] = w.y; sv[2] = w.z; sv[3] = w.w;
+      const uint4 w = lds128(pa + u * US);
+      sv[b] = w.x; sv[b + 1] = w.y; sv[b + 2] = w.z; sv[b + 3] = w.w;
     } else if constexpr (UB == 8) {
-      const uint2 x = *reinterpret_cast<const uint2*>(pa + u * 8);
-      const uint2 y = *reinterpret_cast<const uint2*>(pb + u * 8);
+      const uint2 x = lds64(pa + u * US);
+      const uint2 y = lds64(pb + u * US);
 #pragma unroll
-      for (int j = 0; j < 8; ++j) sv[j] = prmt(j < 4 ? x.x : x.y, j < 4 ? y.x : y.y, pair_sel(j & 3));
+      for (int j = 0; j < 8; ++j) sv[b + j] = prmt(j < 4 ? x.x : x.y, j < 4 ? y.x : y.y, pair_sel(j & 3));
     } else {
-      const uint32_t x = *reinterpret_cast<const uint32_t*>(pa + u * 4);
-      const uint32_t y = *reinterpret_cast<const uint32_t*>(pb + u * 4);
+      constexpr bool IL = US > 8;
+      const int off = IL ? (u >> 1) * US + (u & 1) * 4 : u * 4;
+      const uint32_t x = lds32(pa + off);
+      const uint32_t y = lds32(pb + off);
 #pragma unroll
-      for (int j = 0; j < 4; ++j) sv[j] = prmt(x, y, pair_sel(j));
-    }
-#pragma unroll
-    for (int j = 0; j < UB; ++j) {
-      const int r = u * UB + j;
-      // Eq. (2): H = max(D, E, F) with D = Hdiag + S; E, F >= 0 so the 0 term is
-      // implied.  D goes to the FMA pipe (VIADD.16x2) and feeds both the 3-input
-      // max (VIMNMX3) and the running maximum: max over all D = max over all H
-      // (E and F never exceed an earlier H), so the ALU pipe carries only
-      // 1 + 1 + 1 + 1/2 = 3.5 ops per cell pair.
-      const uint32_t dg = __vadd2(hd, sv[j]);
-      const uint32_t h = __vimax3_s16x2(dg, E[r], F);
-      hd = Hin[r];
-      Hout[r] = h;
-      const uint32_t t = __vadd2(h, nGsGe);                              // H - Gs - Ge
-      E[r] = __viaddmax_s16x2_relu(E[r], nGe, t);                        // Eq. (3)
-      F = __viaddmax_s16x2_relu(F, nGe, t);                              // Eq. (4)
-      if (r & 1) best = __vimax3_s16x2(best, dprev, dg);
-      else dprev = dg;
+      for (int j = 0; j < 4; ++j) sv[b + j] = prmt(x, y, pair_sel(j));
     }
   }
-  Hio = Hout[R1 - 1];
+  uint32_t F = Fio;
+  uint32_t dcur = __vadd2(hdiag, sv[0]);  // D of row R0: H_{R0-1, j-1} + S
+  hdiag = Hio;
+  uint32_t dprev = 0;
+#pragma unroll
+  for (int i = 0; i < N; ++i) {
+    const int r = R0 + i;
+    uint32_t dnext = 0;
+    if (i + 1 < N) dnext = __vadd2(H[r], sv[i + 1]);  // reads H_{r, j-1} before it is replaced
+    const uint32_t h = __vimax3_s16x2(dcur, E[r], F);   // Eq. (2) (E, F >= 0)
+    H[r] = h;
+    const uint32_t t = __vadd2(h, nGsGe);               // H - Gs - Ge
+    E[r] = __viaddmax_s16x2_relu(E[r], nGe, t);         // Eq. (3)
+    F = __viaddmax_s16x2_relu(F, nGe, t);               // Eq. (4)
+    if (r & 1) best = __vimax3_s16x2(best, dprev, dcur);  // max over D = max over H
+    else dprev = dcur;
+    dcur = dnext;
+  }
+  Hio = H[R1 - 1];
   Fio = F;
 }
 

@@ -46,10 +46,21 @@ struct ProfGeom {
   int NL;          // letters = alpha + 1 (PAD = alpha)
   int SB;          // bytes per strip (multiple of 16)
   int n_strips;    // ceil(m / (G*R))
+  int UB;          // bytes per load unit (8 or 4)
+  int il;          // 1: unit-interleaved [letter][unit][lane][UB] (long mode); 0: [letter][lane][LB]
 };
 
 constexpr int LONG_R = 16;   // rows per lane of the intra-task (long pair) geometry, G = 32;
-                             // lane block = LONG_R bytes (no bank padding: 8 strip slots must fit in smem)
+                             // profile unit-interleaved ([letter][unit][lane][8 B]): dense and
+                             // bank-conflict-free (the 16 lanes of an LDS.64 phase hit 16 distinct
+                             // 8-byte slots whatever letters they read)
+#ifndef SW_LONG_IL
+#define SW_LONG_IL 1
+#endif
+#ifndef SW_SMEM_UNION
+#define SW_SMEM_UNION 1
+#endif
+constexpr int LONG_US = SW_LONG_IL ? 32 * 8 : 8;  // bytes between a lane's consecutive 8-byte units in the long profile
 
 // Per-query descriptor of a multi-query launch (processing order: longest first).
 struct QueryDesc {
@@ -94,6 +105,11 @@ struct InterArgs {
   const int2* item_map;      // short item -> (slot, chunk), longest critical path first
   int SB, LS, LB;            // short geometry (G, R of the launch), mode 0 profile
   int SB2, LS2, LB2;         // mode 1 (query-pair) profile
+  // Bank-spread copies of the short strip profile in shared memory: lane group g
+  // reads copy g % ncopy at byte offset (g % ncopy) * cstride; cstride is
+  // 128/ncopy modulo 128, so the groups of one shared-memory phase (random
+  // letters each) hit disjoint banks.  Index 0: mode 0, index 1: mode 1.
+  int ncopy[2], cstride[2];
   int SBL, LSL, LBL;         // long geometry (32 lanes x LONG_R rows)
   int n_long_items;          // sum over queries of n_long * n_super
   uint2* links;              // [gridDim][NT/32][lcap] strip-to-strip rows inside a CTA (long items)
@@ -143,7 +159,7 @@ cudaError_t launch_build_profile(const uint8_t* q, int m, const int8_t* matrix, 
                                  const ProfGeom& g, uint8_t* prof, cudaStream_t st);
 // query-pair profile: word = S[qa_i][a] (low 16) | S[qb_i][a] << 16, lane block LB2
 cudaError_t launch_build_profile_q2(const uint8_t* qa, int ma, const uint8_t* qb, int mb, const int8_t* matrix,
-                                    int alpha, int G, int R, int LB2, int n_strips, int SB2, uint8_t* prof,
+                                    int alpha, int G, int R, int LB2, int LS2, int n_strips, int SB2, uint8_t* prof,
                                     cudaStream_t st);
 int inter_max_ctas_per_sm(int G, int R, int NT, int smem_bytes);
 cudaError_t launch_inter(int G, int R, int NT, int grid, int smem_bytes, const InterArgs& a, cudaStream_t st);

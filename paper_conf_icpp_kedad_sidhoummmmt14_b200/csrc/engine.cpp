@@ -94,6 +94,7 @@ struct sw_handle_s {
   DevBuf glinks, gflags;  // superstrip boundary rows and their counters (long pairs)
   DevBuf rgrows, rflags;  // re-score: CTA-to-CTA rows, counters
   DevBuf imap;            // short work item order
+  DevBuf vq, sinfo;       // packed mode-1 slots: strip-padded query codes per half, per-strip info
   int* pinned_count = nullptr;
   cudaEvent_t ev_begin = nullptr, ev_end = nullptr;
   bool search_timed = false;
@@ -103,6 +104,7 @@ struct sw_handle_s {
   int64_t opt_thr = 0, opt_G = 0, opt_R = 0;
   int64_t opt_t_long = -1;      // >= 0: pairs longer than this always use the intra-task mode
   int64_t opt_query_pairs = 1;  // pair queries two per register for the short pairs
+  int64_t opt_pack_queries = 1; // mode-1 slots: fill the shorter half with further queries (strip-aligned)
   int64_t opt_bank_copy = 1;    // query-pair profile: second smem copy shifted by 64 B for odd lane groups
   int64_t opt_pack_long = 0;    // 1: several long pairs per CTA item when a query has fewer strips than warps
   // last-search bookkeeping
@@ -245,6 +247,8 @@ int32_t sw_set_option(sw_handle_t h, const char* key, int64_t value) {
     h->opt_t_long = value;
   } else if (k == "pack_long") {
     h->opt_pack_long = value;
+  } else if (k == "pack_queries") {
+    h->opt_pack_queries = value;
   } else if (k == "bank_copy") {
     h->opt_bank_copy = value;
   } else if (k == "query_pairs") {
@@ -379,16 +383,13 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
   std::stable_sort(order.begin(), order.end(), [&](int x, int y) { return qlen[size_t(x)] > qlen[size_t(y)]; });
   std::vector<int> ms;
   for (int i : order) ms.push_back(int(qlen[size_t(i)]));
-  // short-pair slots: neighbours in length order form query pairs (mode 1)
-  struct Slot { int mode, k0, k1, nlong; };
-  std::vector<Slot> slots;
+  // geometry from the plain neighbour pairing (mode 1: two queries per register)
   const bool pairs_on = h->opt_query_pairs != 0;
-  for (size_t k = 0; k < order.size();) {
-    if (pairs_on && k + 1 < order.size()) { slots.push_back({1, int(k), int(k + 1), 0}); k += 2; }
-    else { slots.push_back({0, int(k), -1, 0}); k += 1; }
-  }
   std::vector<std::pair<int, int>> slot_m;
-  for (auto& sl : slots) slot_m.push_back({ms[size_t(sl.k0)], sl.mode});
+  for (size_t k = 0; k < order.size();) {
+    if (pairs_on && k + 1 < order.size()) { slot_m.push_back({ms[k], 1}); k += 2; }
+    else { slot_m.push_back({ms[k], 0}); k += 1; }
+  }
   const int nshort_db = np - db->n_long;  // (only for the geometry cost model)
   int G = 4, R = 24;
   choose_geom(h, slot_m, nshort_db > 0 ? db->sum_short_len / nshort_db : 1.0, G, R);
@@ -415,10 +416,51 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
     while (lo < hi) { const int mid = (lo + hi) / 2; if (db->pairs[size_t(mid)].len > Lc) lo = mid + 1; else hi = mid; }
     return lo;
   };
+  // Short-pair slots.  Mode 1: half A (low) and half B (high) each hold a list
+  // of queries laid end to end on strip boundaries; the slot runs max(strips A,
+  // strips B) strips.  The longest unplaced query opens a slot as half A and
+  // half B takes the subset of the remaining queries whose strips best fill it
+  // (subset sum), so the shorter half carries further queries instead of PAD
+  // rows.  A last odd query runs alone in mode 0 (two DB sequences per register).
+  struct Slot { int mode; std::vector<int> A, B; int strips, nlong; };
+  std::vector<Slot> slots;
+  {
+    auto nst = [&](int k) { return std::max(1, (ms[size_t(k)] + G * R - 1) / (G * R)); };
+    std::vector<int> rem;
+    for (size_t k = 0; k < order.size(); ++k) rem.push_back(int(k));  // longest first
+    while (pairs_on && rem.size() >= 2) {
+      const int a0 = rem[0];
+      rem.erase(rem.begin());
+      const int target = nst(a0);
+      std::vector<int> B;
+      if (h->opt_pack_queries && double(rem.size()) * target <= 4e6) {
+        // best subset sum <= target over rem (0/1 knapsack on strip counts)
+        const size_t n = rem.size();
+        std::vector<std::vector<char>> take(n, std::vector<char>(size_t(target) + 1, 0));
+        std::vector<int> bestv(size_t(target) + 1, -1);
+        bestv[0] = 0;
+        for (size_t i = 0; i < n; ++i) {
+          const int w = nst(rem[i]);
+          for (int v = target; v >= w; --v)
+            if (bestv[size_t(v - w)] >= 0 && bestv[size_t(v)] < 0) { bestv[size_t(v)] = 1; take[i][size_t(v)] = 1; }
+        }
+        int v = target;
+        while (v > 0 && bestv[size_t(v)] < 0) --v;
+        for (size_t i = n; i-- > 0 && v > 0;)
+          if (take[i][size_t(v)]) { B.push_back(rem[i]); v -= nst(rem[i]); }
+      } else {
+        B.push_back(rem[0]);  // plain neighbour pairing
+      }
+      std::sort(B.begin(), B.end());
+      for (int b : B) rem.erase(std::find(rem.begin(), rem.end(), b));
+      slots.push_back({1, {a0}, B, target, 0});
+    }
+    for (int k : rem) slots.push_back({0, {k}, {}, nst(k), 0});
+  }
   const int VG = G * (R % 8 == 0 ? 2 : 1);
   double group_steps = 0;  // wavefront steps of all short work if nothing went long
   for (auto& sl : slots) {
-    const int strips = std::max(1, (ms[size_t(sl.k0)] + G * R - 1) / (G * R));
+    const int strips = sl.strips;
     const double seqs = sl.mode == 1 ? 2.0 * np : double(np);
     const double cols = sl.mode == 1 ? 2.0 * db->len_prefix[size_t(np)] : double(db->len_prefix[size_t(np)]);
     group_steps += double(strips) * (cols + seqs * VG);
@@ -437,15 +479,15 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
   }
   int nlong_max = 0;
   for (auto& sl : slots) {
-    const int strips = std::max(1, (ms[size_t(sl.k0)] + G * R - 1) / (G * R));
+    const int strips = sl.strips;
     const int64_t Lc = int64_t(crit / strips);
     sl.nlong = std::max(nlong_opt, pairs_longer_than(Lc));
     nlong_max = std::max(nlong_max, sl.nlong);
   }
   std::vector<int> qnlong(order.size(), 0);
   for (auto& sl : slots) {
-    qnlong[size_t(sl.k0)] = sl.nlong;
-    if (sl.k1 >= 0) qnlong[size_t(sl.k1)] = sl.nlong;
+    for (int k : sl.A) qnlong[size_t(k)] = sl.nlong;
+    for (int k : sl.B) qnlong[size_t(k)] = sl.nlong;
   }
   // profiles: long geometry per query; short geometry per slot
   size_t total = 0;
@@ -460,7 +502,7 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
   std::vector<size_t> off_s;
   std::vector<int> strips_s;
   for (auto& sl : slots) {
-    const int n = std::max(1, (ms[size_t(sl.k0)] + G * R - 1) / (G * R));  // k0 is the longer query
+    const int n = sl.strips;
     strips_s.push_back(n);
     off_s.push_back(total);
     if (sl.nlong < np) total += size_t(n) * (sl.mode == 1 ? SB2 : g1.SB);
@@ -514,6 +556,17 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
   std::vector<SlotDesc> sdesc(slots.size());
   int item = 0;
   int min_pb = np;
+  // packed halves: strip-padded code arrays (PAD = alpha) and per-strip info
+  size_t vq_total = 0, si_total = 0;
+  for (auto& sl : slots)
+    if (sl.mode == 1) { vq_total += 2 * size_t(sl.strips) * G * R; si_total += size_t(sl.strips); }
+  std::vector<StripInfo> sinfo(si_total);
+  if (vq_total) {
+    SW_CK(h->vq.ensure(vq_total));
+    SW_CK(cudaMemsetAsync(h->vq.p, alpha, vq_total, c.st));
+    SW_CK(h->sinfo.ensure(si_total * sizeof(StripInfo)));
+  }
+  size_t vq_off = 0, si_off = 0;
   for (size_t j = 0; j < slots.size(); ++j) {
     const Slot& sl = slots[j];
     SlotDesc& d = sdesc[j];
@@ -521,10 +574,37 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
     d.prof = prof + off_s[j];
     d.mode = sl.mode;
     d.n_strips = strips_s[j];
-    d.qidx0 = order[size_t(sl.k0)];
+    d.qidx0 = order[size_t(sl.A[0])];
     d.scores0 = c.dscores + int64_t(d.qidx0) * db->n_seqs;
-    d.qidx1 = sl.mode == 1 ? order[size_t(sl.k1)] : -1;
-    d.scores1 = sl.mode == 1 ? c.dscores + int64_t(d.qidx1) * db->n_seqs : nullptr;
+    d.qidx1 = -1;
+    d.scores1 = nullptr;
+    d.sinfo = nullptr;
+    uint8_t* vA = nullptr;
+    uint8_t* vB = nullptr;
+    if (sl.mode == 1) {
+      const size_t GR = size_t(G) * R;
+      vA = h->vq.as<uint8_t>() + vq_off;
+      vB = vA + size_t(sl.strips) * GR;
+      vq_off += 2 * size_t(sl.strips) * GR;
+      StripInfo* si = sinfo.data() + si_off;
+      d.sinfo = h->sinfo.as<StripInfo>() + si_off;
+      si_off += size_t(sl.strips);
+      for (int s0 = 0; s0 < sl.strips; ++s0) si[s0] = StripInfo{0xffffffffu, -1, -1, 0};
+      for (int hf = 0; hf < 2; ++hf) {
+        const std::vector<int>& L = hf == 0 ? sl.A : sl.B;
+        uint8_t* dst = hf == 0 ? vA : vB;
+        int st0 = 0;
+        for (int kq : L) {
+          const int n = std::max(1, (ms[size_t(kq)] + G * R - 1) / (G * R));
+          if (ms[size_t(kq)] > 0)
+            SW_CK(cudaMemcpyAsync(dst + size_t(st0) * GR, qptr(kq), size_t(ms[size_t(kq)]), cudaMemcpyDeviceToDevice,
+                                  c.st));
+          if (st0 > 0) si[st0].keep &= hf == 0 ? 0xffff0000u : 0x0000ffffu;  // new query: zero boundary
+          (hf == 0 ? si[st0 + n - 1].emit0 : si[st0 + n - 1].emit1) = order[size_t(kq)];
+          st0 += n;
+        }
+      }
+    }
     d.pair_begin = sl.nlong;
     d.item_begin = item;
     d.n_items = ns > 0 ? (sl.mode == 1 ? (2 * ns + NG - 1) / NG : (ns + NG - 1) / NG) : 0;
@@ -533,13 +613,14 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
       min_pb = std::min(min_pb, sl.nlong);
       const double sumS = pair_len_sum(sl.nlong, np) + double(ns) * 2 * G;
       if (sl.mode == 1) {
-        SW_CK(launch_build_profile_q2(qptr(sl.k0), ms[size_t(sl.k0)], qptr(sl.k1), ms[size_t(sl.k1)], dmat, alpha,
-                                      G, R, LB2, LS2, d.n_strips, SB2, prof + off_s[j], c.st));
+        const int rows = sl.strips * G * R;
+        SW_CK(launch_build_profile_q2(vA, rows, vB, rows, dmat, alpha, G, R, LB2, LS2, d.n_strips, SB2,
+                                      prof + off_s[j], c.st));
         cells_computed += 2.0 * (2.0 * sumS) * double(d.n_strips) * G * R;  // every sequence, 2 queries
       } else {
         ProfGeom gq = g1;
         gq.n_strips = d.n_strips;
-        SW_CK(launch_build_profile(qptr(sl.k0), ms[size_t(sl.k0)], dmat, alpha, gq, prof + off_s[j], c.st));
+        SW_CK(launch_build_profile(qptr(sl.A[0]), ms[size_t(sl.A[0])], dmat, alpha, gq, prof + off_s[j], c.st));
         cells_computed += 2.0 * sumS * double(d.n_strips) * G * R;
       }
       ++launches;
@@ -572,6 +653,8 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
       }
     }
   }
+  if (si_total)
+    SW_CK(cudaMemcpyAsync(h->sinfo.p, sinfo.data(), si_total * sizeof(StripInfo), cudaMemcpyHostToDevice, c.st));
   SW_CK(h->imap.ensure(std::max<size_t>(imap.size(), 1) * sizeof(int2)));
   if (!imap.empty())
     SW_CK(cudaMemcpyAsync(h->imap.p, imap.data(), imap.size() * sizeof(int2), cudaMemcpyHostToDevice, c.st));
@@ -641,6 +724,8 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
   a.bbuf = (max_strips > 1 && min_pb < np) ? h->bbuf.as<uint2>() : nullptr;
   a.bcap = bcap;
   a.work_counter = h->counters.as<int>();
+  a.scores_all = c.dscores;
+  a.n_seqs = db->n_seqs;
   a.thr = c.thr;
   a.ovf = c.ovf;
   a.ovf_count = c.ovf_count;

@@ -28,6 +28,9 @@ constexpr int8_t PAD_SCORE = -64;  // S[.][PAD] = S[PAD][.] <= 0 (reading R-12)
 // producer is this many columns ahead, so producer and consumer warps of a
 // chain run decoupled instead of in lock-step (the consumer then rarely waits).
 constexpr int LINK_LAG = 64;
+#ifndef SW_DUAL
+#define SW_DUAL 1  // both sub-lanes in one interleaved row sweep (gotoh_rows_dual)
+#endif
 constexpr int RESCORE_LAG = 16;  // re-score chains: one round per CTA, short lag keeps the critical path short
 
 // ---------------------------------------------------------------------------
@@ -91,8 +94,10 @@ __global__ void build_profile_q2_kernel(const uint8_t* __restrict__ qa, int ma, 
       const int r = (rr - k * LB2) / 4;
       if (k < G && r < R) {
         const int row = s * G * R + k * R + r;
-        const int va = (row < ma && a < alpha) ? M[qa[row] * alpha + a] : PAD_SCORE;
-        const int vb = (row < mb && a < alpha) ? M[qb[row] * alpha + a] : PAD_SCORE;
+        // rows past a query, and PAD codes (= alpha) that pad packed queries to whole strips
+        const int ca = row < ma ? qa[row] : alpha, cb = row < mb ? qb[row] : alpha;
+        const int va = (ca < alpha && a < alpha) ? M[ca * alpha + a] : PAD_SCORE;
+        const int vb = (cb < alpha && a < alpha) ? M[cb * alpha + a] : PAD_SCORE;
         v = (uint32_t(va) & 0xffffu) | (uint32_t(vb) << 16);
       }
     }
@@ -259,9 +264,13 @@ __device__ __forceinline__ void strip_pass(const uint8_t* sprof, int LS, int LB,
       }
       if constexpr (V == 2) {
         uint32_t h1 = cH, f1 = cF;
-        // sub-lane 1 (rows RH..R-1, column t-1) first: it reads rows it owns only
-        gotoh_rows_inplace<R, RH, R, Q2, US>(HA, E, best, hdiag1, ppa, ppb, h1, f1, nGe, nGsGe);
-        gotoh_rows_inplace<R, 0, RH, Q2, US>(HA, E, best, hdiag, pa, pb, rH, rF, nGe, nGsGe);
+        if constexpr (SW_DUAL && Q2) {  // measured: +3% for the query-pair mode, -2% with the PRMT (mode 0)
+          gotoh_rows_dual<R, Q2, US>(HA, E, best, hdiag, pa, pb, rH, rF, hdiag1, ppa, ppb, h1, f1, nGe, nGsGe);
+        } else {
+          // sub-lane 1 (rows RH..R-1, column t-1) first: it reads rows it owns only
+          gotoh_rows_inplace<R, RH, R, Q2, US>(HA, E, best, hdiag1, ppa, ppb, h1, f1, nGe, nGsGe);
+          gotoh_rows_inplace<R, 0, RH, Q2, US>(HA, E, best, hdiag, pa, pb, rH, rF, nGe, nGsGe);
+        }
         cH = rH;
         cF = rF;
         ppa = pa;
@@ -518,31 +527,53 @@ __global__ void __launch_bounds__(NT) inter_kernel(InterArgs a) {
           __syncthreads();
           loaded = want;
         }
-        if (q2)
-          strip_pass<G, R, false, true>(gprof, a.LS2, a.LB2, a.stream + pr.off, pr.len, T, k, s > 0,
+        if (q2) {
+          const StripInfo si = d.sinfo[s];
+          const bool rd = s > 0 && si.keep != 0;
+          if (rd && si.keep != FULL) {  // one half starts a new query: zero its half of the boundary row
+            for (int c = k; c < T; c += G) {
+              const uint2 v = bb[c];
+              bb[c] = make_uint2(v.x & si.keep, v.y & si.keep);
+            }
+            __syncwarp();
+          }
+          strip_pass<G, R, false, true>(gprof, a.LS2, a.LB2, a.stream + pr.off, pr.len, T, k, rd,
                                         s + 1 < d.n_strips, bb, bb, Link{}, a.code_pad2,
                                         a.nGe, a.nGsGe, best, half ? 8u : 0u);
-        else
-          strip_pass<G, R, false>(gprof, a.LS, a.LB, a.stream + pr.off, pr.len, T, k, s > 0, s + 1 < d.n_strips,
-                                  bb, bb, Link{}, a.code_pad2, a.nGe, a.nGsGe, best);
-      }
+          if (si.emit0 >= 0 || si.emit1 >= 0) {  // a query of either half ends with this strip
+            uint32_t bg = best;
 #pragma unroll
-      for (int o = G / 2; o > 0; o >>= 1) best = __vmaxs2(best, __shfl_xor_sync(FULL, best, o, G));
-      if (valid && k == 0) {
-        if (q2) {
-          const int id = half ? pr.id1 : pr.id0;
-          const int v0 = int(int16_t(best & 0xffffu)), v1 = int(int16_t(best >> 16));
-          d.scores0[id] = v0;
-          d.scores1[id] = v1;
-          if (v0 >= a.thr) {
-            const int e = atomicAdd(a.ovf_count, 1);
-            if (e < a.ovf_cap) a.ovf[e] = OvfRec{d.qidx0, p, half, 0};
-          }
-          if (v1 >= a.thr) {
-            const int e = atomicAdd(a.ovf_count, 1);
-            if (e < a.ovf_cap) a.ovf[e] = OvfRec{d.qidx1, p, half, 0};
+            for (int o = G / 2; o > 0; o >>= 1) bg = __vmaxs2(bg, __shfl_xor_sync(FULL, bg, o, G));
+            if (valid && k == 0) {
+              const int id = half ? pr.id1 : pr.id0;
+              if (si.emit0 >= 0) {
+                const int v = int(int16_t(bg & 0xffffu));
+                a.scores_all[(int64_t)si.emit0 * a.n_seqs + id] = v;
+                if (v >= a.thr) {
+                  const int e = atomicAdd(a.ovf_count, 1);
+                  if (e < a.ovf_cap) a.ovf[e] = OvfRec{si.emit0, p, half, 0};
+                }
+              }
+              if (si.emit1 >= 0) {
+                const int v = int(int16_t(bg >> 16));
+                a.scores_all[(int64_t)si.emit1 * a.n_seqs + id] = v;
+                if (v >= a.thr) {
+                  const int e = atomicAdd(a.ovf_count, 1);
+                  if (e < a.ovf_cap) a.ovf[e] = OvfRec{si.emit1, p, half, 0};
+                }
+              }
+            }
+            best &= (si.emit0 >= 0 ? 0xffff0000u : 0xffffffffu) & (si.emit1 >= 0 ? 0x0000ffffu : 0xffffffffu);
           }
         } else {
+          strip_pass<G, R, false>(gprof, a.LS, a.LB, a.stream + pr.off, pr.len, T, k, s > 0, s + 1 < d.n_strips,
+                                  bb, bb, Link{}, a.code_pad2, a.nGe, a.nGsGe, best);
+        }
+      }
+      if (!q2) {  // mode 0: one query, both halves are DB sequences
+#pragma unroll
+        for (int o = G / 2; o > 0; o >>= 1) best = __vmaxs2(best, __shfl_xor_sync(FULL, best, o, G));
+        if (valid && k == 0) {
           QueryDesc qd;
           qd.scores = d.scores0;
           qd.qidx = d.qidx0;

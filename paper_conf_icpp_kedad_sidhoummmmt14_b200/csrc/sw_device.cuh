@@ -130,6 +130,81 @@ __device__ __forceinline__ void gotoh_rows_inplace(uint32_t (&H)[R], uint32_t (&
   Fio = F;
 }
 
+// Profile values S(q_r, letter) of rows [R0, R1) for one lane (see gotoh_rows_inplace).
+template <int R, int R0, int R1, bool Q2, int US>
+__device__ __forceinline__ void load_rows(uint32_t (&sv)[R1 - R0], uint32_t pa, uint32_t pb) {
+  constexpr int N = R1 - R0;
+  constexpr int UB = Q2 ? 4 : ((R % 8 == 0 && R0 % 8 == 0 && N % 8 == 0) ? 8 : 4);
+#pragma unroll
+  for (int u = R0 / UB; u < R1 / UB; ++u) {
+    const int b = u * UB - R0;
+    if constexpr (Q2) {
+      const uint4 w = lds128(pa + u * US);
+      sv[b] = w.x; sv[b + 1] = w.y; sv[b + 2] = w.z; sv[b + 3] = w.w;
+    } else if constexpr (UB == 8) {
+      const uint2 x = lds64(pa + u * US);
+      const uint2 y = lds64(pb + u * US);
+#pragma unroll
+      for (int j = 0; j < 8; ++j) sv[b + j] = prmt(j < 4 ? x.x : x.y, j < 4 ? y.x : y.y, pair_sel(j & 3));
+    } else {
+      constexpr bool IL = US > 8;
+      const int off = IL ? (u >> 1) * US + (u & 1) * 4 : u * 4;
+      const uint32_t x = lds32(pa + off);
+      const uint32_t y = lds32(pb + off);
+#pragma unroll
+      for (int j = 0; j < 4; ++j) sv[b + j] = prmt(x, y, pair_sel(j));
+    }
+  }
+}
+
+// Both sub-lanes of a lane in one interleaved sweep: sub-lane 0 = rows [0, RH)
+// of column t, sub-lane 1 = rows [RH, R) of column t-1 (its inputs hdiag1 /
+// Hio1 / Fio1 are sub-lane 0's outputs of the previous step).  The two F
+// chains are independent, so emitting their rows alternately hands the
+// scheduler two ready instructions per dependency step.
+template <int R, bool Q2, int US>
+__device__ __forceinline__ void gotoh_rows_dual(uint32_t (&H)[R], uint32_t (&E)[R], uint32_t& best,
+                                                uint32_t& hdiag0, uint32_t pa0, uint32_t pb0, uint32_t& Hio0,
+                                                uint32_t& Fio0, uint32_t& hdiag1, uint32_t pa1, uint32_t pb1,
+                                                uint32_t& Hio1, uint32_t& Fio1, uint32_t nGe, uint32_t nGsGe) {
+  constexpr int RH = R / 2;
+  static_assert(R % 8 == 0, "two sub-lanes of whole 4-row units");
+  uint32_t s0[RH], s1[RH];
+  load_rows<R, 0, RH, Q2, US>(s0, pa0, pb0);
+  load_rows<R, RH, R, Q2, US>(s1, pa1, pb1);
+  uint32_t F0 = Fio0, F1 = Fio1;
+  uint32_t d0 = __vadd2(hdiag0, s0[0]);
+  uint32_t d1 = __vadd2(hdiag1, s1[0]);
+  hdiag0 = Hio0;
+  hdiag1 = Hio1;
+#pragma unroll
+  for (int i = 0; i < RH; ++i) {
+    const int r0 = i, r1 = RH + i;
+    uint32_t n0 = 0, n1 = 0;
+    if (i + 1 < RH) {  // next rows' diagonals read H_{r, j-1} before it is replaced
+      n0 = __vadd2(H[r0], s0[i + 1]);
+      n1 = __vadd2(H[r1], s1[i + 1]);
+    }
+    const uint32_t h0 = __vimax3_s16x2(d0, E[r0], F0);  // Eq. (2)
+    const uint32_t h1 = __vimax3_s16x2(d1, E[r1], F1);
+    H[r0] = h0;
+    H[r1] = h1;
+    const uint32_t t0 = __vadd2(h0, nGsGe);
+    const uint32_t t1 = __vadd2(h1, nGsGe);
+    E[r0] = __viaddmax_s16x2_relu(E[r0], nGe, t0);    // Eq. (3)
+    E[r1] = __viaddmax_s16x2_relu(E[r1], nGe, t1);
+    F0 = __viaddmax_s16x2_relu(F0, nGe, t0);          // Eq. (4)
+    F1 = __viaddmax_s16x2_relu(F1, nGe, t1);
+    best = __vimax3_s16x2(best, d0, d1);              // max over D = max over H
+    d0 = n0;
+    d1 = n1;
+  }
+  Hio0 = H[RH - 1];
+  Fio0 = F0;
+  Hio1 = H[R - 1];
+  Fio1 = F1;
+}
+
 // Lane block of the query-pair profile: R 4-byte rows, rounded to an odd number
 // of 16-byte units (bank-conflict-free LDS.128 across the 8 lanes of a phase).
 __host__ __device__ constexpr int lane_block_bytes_q2(int R) { return (((R / 4) | 1) * 16); }

@@ -83,7 +83,18 @@ struct QueryDesc {
 // Short-pair work of one "slot": a single query (mode 0: two DB sequences per
 // s16x2 register, int8 profile) or a query PAIR (mode 1: two queries per
 // register, one DB sequence per lane group, s16x2 profile).
+// Mode-1 slots pack several queries per s16x2 half, each starting on a strip
+// boundary (fills the shorter half of a query pair with
+// further short queries instead of PAD rows).  Per strip of such a slot:
+struct StripInfo {
+  uint32_t keep;             // halves that continue the query of the previous strip (0x0000ffff: low
+                             // half, 0xffff0000: high half); a new query starts from a zero boundary row
+  int32_t emit0, emit1;      // query whose last strip this is, per half (-1: none)
+  int32_t pad_;
+};
+
 struct SlotDesc {
+  const StripInfo* sinfo;    // mode 1: [n_strips]
   const uint8_t* prof;       // mode 0: [n_strips][SB] int8; mode 1: [n_strips][SB2] s16x2
   int32_t* scores0;          // scores row of the (first) query
   int32_t* scores1;          // mode 1: row of the second query
@@ -124,6 +135,8 @@ struct InterArgs {
   uint2* bbuf;               // boundary rows of multi-strip short items, [gridDim][NG][bcap]
   int bcap;
   int* work_counter;
+  int32_t* scores_all;       // [n_queries (caller order)][n_seqs]: mode-1 emission target
+  int64_t n_seqs;
   int32_t thr;               // overflow threshold (int16 max >= thr -> re-score)
   OvfRec* ovf;
   int* ovf_count;

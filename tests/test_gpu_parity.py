@@ -240,3 +240,22 @@ def test_query_pairing_modes(pairs):
     qc, qo = _seqs([700, 31, 256, 255, 1, 90, 400], rng)
     got = gpu_scores(qc, qo, dc, do, opts={"query_pairs": pairs})
     np.testing.assert_array_equal(got, oracle_scores(qc, qo, dc, do))
+
+
+@pytest.mark.parametrize("pack", [0, 1])
+@pytest.mark.parametrize("thr", [0, 40])
+def test_query_packing(pack, thr):
+    """Mode-1 slots whose shorter half carries several queries laid end to end on
+    strip boundaries (a new query starts from a zero boundary row; each query's
+    score is emitted at its last strip).  thr > 0 forces the int32 re-score of
+    packed queries' pairs (the flag must name the right query)."""
+    rng = np.random.default_rng(41 + pack + thr)
+    dc, do = _seqs(list(rng.integers(1, 500, size=120)) + [0, 1, 4], rng)
+    # strips at G*R = 96: 1900 -> 20, 1100 -> 12, 500 -> 6, 190 -> 2, ...
+    ql = [1900, 1100, 500, 190, 96, 97, 5, 1, 800, 380, 33]
+    qc, qo = _seqs(ql, rng)
+    opts = {"pack_queries": pack, "force_G": 4, "force_R": 24}
+    if thr:
+        opts["overflow_threshold"] = thr
+    got = gpu_scores(qc, qo, dc, do, opts=opts)
+    np.testing.assert_array_equal(got, oracle_scores(qc, qo, dc, do))

@@ -13,6 +13,8 @@ reps = int(os.environ.get("PROF_REPS", "2"))
 wl = os.environ.get("PROF_WORKLOAD", "c2")
 c = swgen.make_config(wl, n_db=int(os.environ["PROF_NDB"]) if os.environ.get("PROF_NDB") else None)
 h = sw.Handle(0)
+for kv in filter(None, os.environ.get("SWDUAL_OPTS", "").split(",")):
+    h.set_option(kv.split("=")[0], int(kv.split("=")[1]))
 for k in ("force_G", "force_R"):
     if os.environ.get(k.upper()):
         h.set_option(k, int(os.environ[k.upper()]))

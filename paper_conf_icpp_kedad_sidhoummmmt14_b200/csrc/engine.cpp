@@ -681,7 +681,7 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
   const int grid = int(std::max<int64_t>(1, std::min<int64_t>(n_items, int64_t(occ) * h->sms)));
   const int32_t max_short = min_pb < np ? db->pairs[size_t(min_pb)].len : 0;
   const int32_t max_long = db->pairs[0].len;
-  const int bcap = max_short + 4 * G + 8;  // wave width up to V*G sub-lanes (V <= 3)
+  const int bcap = ((max_short + 4 * G + 8 + 4) + 3) / 4 * 4;  // wave width up to V*G sub-lanes (V <= 3) + align pad
   if (max_strips > 1 && min_pb < np) SW_CK(h->bbuf.ensure(size_t(grid) * NG * bcap * sizeof(uint2)));
   const int lcap = max_long + 64 + 8;
   if (nlong_max > 0 && max_lstrips > 1) SW_CK(h->bbuf_long.ensure(size_t(grid) * W * lcap * sizeof(uint2)));

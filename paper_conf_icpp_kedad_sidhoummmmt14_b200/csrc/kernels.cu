@@ -28,6 +28,9 @@ constexpr int8_t PAD_SCORE = -64;  // S[.][PAD] = S[PAD][.] <= 0 (reading R-12)
 // producer is this many columns ahead, so producer and consumer warps of a
 // chain run decoupled instead of in lock-step (the consumer then rarely waits).
 constexpr int LINK_LAG = 64;
+#ifndef SW_DUAL_LONG
+#define SW_DUAL_LONG 0
+#endif
 #ifndef SW_DUAL
 #define SW_DUAL 1  // both sub-lanes in one interleaved row sweep (gotoh_rows_dual)
 #endif
@@ -172,6 +175,34 @@ __device__ __forceinline__ void copy_strip(uint8_t* dst, const uint8_t* __restri
   for (int i = threadIdx.x; i < bytes / 16; i += blockDim.x) d[i] = __ldg(s + i);
 }
 
+// DB codes of the current pair: every strip pass of an item re-reads them, so
+// they could stay cached between strips (SW_CODES 0: streaming/evict-first,
+// 1: default caching, 2: L2 evict_last).  Measured on config 3: 1 and 2 cut
+// DRAM reads by 23% but run 1% slower (the kernel is ALU-bound); 0 is kept.
+#ifndef SW_CODES
+#define SW_CODES 0
+#endif
+#ifndef SW_BB_HINT
+#define SW_BB_HINT 0
+#endif
+__device__ __forceinline__ uint4 ld_bb(const uint2* p, uint64_t pol) {
+  if constexpr (SW_BB_HINT) return ld_l2_last(p, pol);
+  else return *reinterpret_cast<const uint4*>(p);
+}
+__device__ __forceinline__ void st_bb(uint2* p, uint2 v, uint64_t pol) {
+  if constexpr (SW_BB_HINT) st_l2_last(p, v, pol);
+  else *p = v;
+}
+__device__ __forceinline__ uint2 ld_codes(const uint2* p, uint64_t pol) {
+  if constexpr (SW_CODES == 0) return __ldcs(p);
+  else if constexpr (SW_CODES == 1) return __ldg(p);
+  else {
+    uint2 v;
+    asm volatile("ld.global.nc.L2::cache_hint.v2.u32 {%0, %1}, [%2], %3;" : "=r"(v.x), "=r"(v.y) : "l"(p), "l"(pol));
+    return v;
+  }
+}
+
 // One strip pass of a lane group over one pair: G lanes x R rows, columns
 // streamed as an anti-diagonal wave.  Boundary rows: lane 0 reads the strip
 // above at rp[c] (c = column, rp = row base + G - 1), lane G-1 writes this
@@ -209,6 +240,9 @@ __device__ __forceinline__ void strip_pass(const uint8_t* sprof, int LS, int LB,
   const uint32_t pad_row = sbase + (code_pad2 & 0xffu) * LS + laneoff;
   uint32_t ppa = pad_row, ppb = pad_row;
   rp += VG - 1;  // sub-lane 0 of lane 0 reads column c at rp[c + VG - 1]
+  // SW_BB_HINT 1: boundary rows with an L2 evict_last policy (DRAM writes -35%
+  // on config 3, but 1% slower: the kernel is ALU-bound, DRAM is ~3% busy)
+  const uint64_t pol = (SW_BB_HINT || SW_CODES == 2) ? l2_evict_last_policy() : 0;
 
   // lane 0 prefetch of block 0: 4 columns of codes and (if rd) 4 boundary cells.
   // L and t0 are multiples of 4, so one compare guards a whole block.
@@ -217,10 +251,13 @@ __device__ __forceinline__ void strip_pass(const uint8_t* sprof, int LS, int LB,
   int seen = -1;
   if (LINKED && rd && L > 0) wait_progress(lk, lk.in_base + min(4 + VG - 1 + LINK_LAG, L + VG), seen);
   if (lead && L > 0) {
-    cw = __ldcs(codes);
+    cw = ld_codes(codes, pol);
     if (rd) {
       if (LINKED) { tb0 = __ldcg(rp + 0); tb1 = __ldcg(rp + 1); tb2 = __ldcg(rp + 2); tb3 = __ldcg(rp + 3); }
-      else { tb0 = rp[0]; tb1 = rp[1]; tb2 = rp[2]; tb3 = rp[3]; }
+      else {  // rp is 32-byte aligned (see the bb base in inter_kernel)
+        const uint4 x = ld_bb(rp, pol), y = ld_bb(rp + 2, pol);
+        tb0 = make_uint2(x.x, x.y); tb1 = make_uint2(x.z, x.w); tb2 = make_uint2(y.x, y.y); tb3 = make_uint2(y.z, y.w);
+      }
     }
   }
   __syncwarp();
@@ -231,10 +268,13 @@ __device__ __forceinline__ void strip_pass(const uint8_t* sprof, int LS, int LB,
     if (LINKED && rd && t0 + 4 < L) wait_progress(lk, lk.in_base + min(t0 + 8 + VG - 1 + LINK_LAG, L + VG), seen);
     if (lead) {
       if (t0 + 4 < L) {
-        cw = __ldcs(codes + ((t0 + 4) >> 2));
+        cw = ld_codes(codes + ((t0 + 4) >> 2), pol);
         if (rd) {
           if (LINKED) { tb0 = __ldcg(rp + 0); tb1 = __ldcg(rp + 1); tb2 = __ldcg(rp + 2); tb3 = __ldcg(rp + 3); }
-          else { tb0 = rp[0]; tb1 = rp[1]; tb2 = rp[2]; tb3 = rp[3]; }
+          else {
+            const uint4 x = ld_bb(rp, pol), y = ld_bb(rp + 2, pol);
+            tb0 = make_uint2(x.x, x.y); tb1 = make_uint2(x.z, x.w); tb2 = make_uint2(y.x, y.y); tb3 = make_uint2(y.z, y.w);
+          }
         }
       } else {
         cw = make_uint2(pad4, pad4);
@@ -264,7 +304,7 @@ __device__ __forceinline__ void strip_pass(const uint8_t* sprof, int LS, int LB,
       }
       if constexpr (V == 2) {
         uint32_t h1 = cH, f1 = cF;
-        if constexpr (SW_DUAL && Q2) {  // measured: +3% for the query-pair mode, -2% with the PRMT (mode 0)
+        if constexpr (SW_DUAL && (Q2 || (SW_DUAL_LONG && LINKED))) {  // measured: +3% for the query-pair mode, -2% with the PRMT (mode 0)
           gotoh_rows_dual<R, Q2, US>(HA, E, best, hdiag, pa, pb, rH, rF, hdiag1, ppa, ppb, h1, f1, nGe, nGsGe);
         } else {
           // sub-lane 1 (rows RH..R-1, column t-1) first: it reads rows it owns only
@@ -287,7 +327,7 @@ __device__ __forceinline__ void strip_pass(const uint8_t* sprof, int LS, int LB,
       }
       if (wr && tail) {
         if (LINKED) __stcg(wp + j, make_uint2(sH, sF));
-        else wp[j] = make_uint2(sH, sF);
+        else st_bb(wp + j, make_uint2(sH, sF), pol);
       }
     }
     wp += 4;
@@ -343,7 +383,9 @@ __global__ void __launch_bounds__(NT) inter_kernel(InterArgs a) {
   const int lane = tid & 31, warp = tid >> 5;
   const int n_long_items = a.n_long_items;
   const int n_items = n_long_items + a.n_short_items;
-  uint2* __restrict__ bb = a.bbuf + ((size_t)blockIdx.x * NG + g) * (size_t)a.bcap;
+  // per-group boundary row; offset so that &bb[V*G - 1] is 32-byte aligned (bcap % 4 == 0)
+  constexpr int BB_PAD = (4 - (G * SubLanes<R>::V - 1) % 4) % 4;
+  uint2* __restrict__ bb = a.bbuf + ((size_t)blockIdx.x * NG + g) * (size_t)a.bcap + BB_PAD;
   int loaded = -1;  // (query rank << 16 | strip) of the short profile in shared memory (CTA-uniform)
 
   for (;;) {

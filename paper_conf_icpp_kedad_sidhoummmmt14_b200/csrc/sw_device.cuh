@@ -44,6 +44,24 @@ __host__ __device__ constexpr int lane_block_bytes(int R) {
   return ((R % 8 == 0) ? (((R / 8) | 1) * 8) : (((R / 4) | 1) * 4));
 }
 
+// Boundary rows of multi-strip lane groups are rewritten and re-read once per
+// strip pass: keep them in L2 (evict_last) while the DB codes stream through
+// with evict-first loads, so they need not travel to DRAM and back.
+__device__ __forceinline__ uint64_t l2_evict_last_policy() {
+  uint64_t p;
+  asm volatile("createpolicy.fractional.L2::evict_last.b64 %0, 1.0;" : "=l"(p));
+  return p;
+}
+__device__ __forceinline__ uint4 ld_l2_last(const void* a, uint64_t pol) {
+  uint4 v;
+  asm volatile("ld.global.L2::cache_hint.v4.u32 {%0, %1, %2, %3}, [%4], %5;"
+               : "=r"(v.x), "=r"(v.y), "=r"(v.z), "=r"(v.w) : "l"(a), "l"(pol));
+  return v;
+}
+__device__ __forceinline__ void st_l2_last(void* a, uint2 v, uint64_t pol) {
+  asm volatile("st.global.L2::cache_hint.v2.u32 [%0], {%1, %2}, %3;" :: "l"(a), "r"(v.x), "r"(v.y), "l"(pol) : "memory");
+}
+
 // Shared-memory loads by 32-bit shared-window address (the profile pointers
 // stay 32-bit: fewer registers than generic 64-bit pointers, no address
 // rematerialisation in the hot loop).

@@ -41,6 +41,8 @@ WORKLOADS = {
     "c2": "BASELINE config 2: 1 query (567 aa) vs Swiss-Prot-sized synthetic DB (570k seqs, ~205M residues), BLOSUM62, gap 10/2",
     "c1": "BASELINE config 1: 1 query (144 aa) vs 1,000 synthetic sequences, BLOSUM62, gap 10/2",
     "c4": "BASELINE config 4: queries 2,000-35,000 aa vs 1,500 long synthetic sequences (>3,000 aa)",
+    "t5hom": "PAPER Table V homogeneous set: 40 queries 4,500-5,000 aa vs Swiss-Prot-sized synthetic DB (570k seqs)",
+    "t5het": "PAPER Table V heterogeneous set: 40 queries 4-35,213 aa vs Swiss-Prot-sized synthetic DB (570k seqs)",
 }
 REASONS = {0x1: "gpu_idle", 0x2: "applications_clocks_setting", 0x4: "sw_power_cap", 0x8: "hw_slowdown",
            0x10: "sync_boost", 0x20: "sw_thermal_slowdown", 0x40: "hw_thermal_slowdown",
@@ -144,7 +146,7 @@ def config_obj(args, c, q_lens, d_lens, n):
             "matrix": "BLOSUM62", "gap_open": 10, "gap_extend": 2,
             "shards": n, "placement": "dual-approximation (query, shard) tasks",
             "l2": "inputs larger than L2: 205 MB packed DB > 126 MB L2, streamed once per query per step"
-            if args.workload in ("c2", "c3") and args.n_db is None else "small workload"}
+            if args.workload in ("c2", "c3", "t5hom", "t5het") and args.n_db is None else "small workload"}
 
 
 def cpu_baseline(c, target_cells: float, seed: int = 2024) -> dict:

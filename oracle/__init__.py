@@ -11,8 +11,8 @@ Only tests/, __graft_entry__.smoke() and bench.py (cpu_baseline leg and
 with it.  Pins: tests/test_oracle_pins.py (brute force, textbook values,
 special cases, invariants, worked goldens under tests/golden/).
 
-Parity status: oracle_gotoh_score / gotoh_search are pinned (see DESIGN.md
-"Oracle pins"); nothing here is "parity unpinned".
+Parity status: oracle_gotoh_score / gotoh_search / gotoh_align are pinned (see
+DESIGN.md "Oracle pins"); nothing here is "parity unpinned".
 """
 from __future__ import annotations
 
@@ -54,6 +54,11 @@ def _load():
             ctypes.c_int64, ctypes.c_int64,
             ctypes.c_void_p, ctypes.c_int32, ctypes.c_int32, ctypes.c_int32,
             ctypes.c_void_p]
+        lib.oracle_gotoh_align.restype = ctypes.c_int32
+        lib.oracle_gotoh_align.argtypes = [
+            ctypes.c_void_p, ctypes.c_int64, ctypes.c_void_p, ctypes.c_int64,
+            ctypes.c_void_p, ctypes.c_int32, ctypes.c_int32, ctypes.c_int32,
+            ctypes.c_void_p, ctypes.c_void_p, ctypes.c_int32]
         _lib = lib
     return _lib
 
@@ -121,3 +126,19 @@ def gotoh_search(qcodes, qoff, dcodes, doff, S, gs: int, ge: int, procs: int = 1
         for b0, b1, blk in pool.imap_unordered(_search_chunk, jobs):
             out[:, b0:b1] = blk
     return out
+
+
+def gotoh_align(q, d, S, gs: int, ge: int):
+    """Best local alignment of one pair (sw_oracle.c oracle_gotoh_align):
+    (score, q_begin, q_end, d_begin, d_end, ops) with ops run-length codes
+    (len << 2 | op), op 0 = M, 1 = I (query vs gap), 2 = D (subject vs gap)."""
+    q = np.ascontiguousarray(np.asarray(q, dtype=np.uint8))
+    d = np.ascontiguousarray(np.asarray(d, dtype=np.uint8))
+    S = _matrix(S)
+    out5 = np.zeros(5, dtype=np.int32)
+    ops = np.zeros(len(q) + len(d) + 1, dtype=np.uint32)
+    n = _load().oracle_gotoh_align(_ptr(q), len(q), _ptr(d), len(d), _ptr(S), S.shape[0], int(gs), int(ge),
+                                   _ptr(out5), _ptr(ops), len(ops))
+    if n < 0:
+        raise ValueError("oracle: bad input (code >= alphabet size or OOM)")
+    return (int(out5[0]), int(out5[1]), int(out5[2]), int(out5[3]), int(out5[4]), [int(x) for x in ops[:n]])

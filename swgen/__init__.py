@@ -143,6 +143,15 @@ CONFIGS = {
                plant_ids=[1.0, 0.95, 0.9]),
     "c5": dict(db_seed=5, n_db=50_000_000, kind=0, mu=5.545, q_seed=3, q_lens=SWEEP,
                plant_ids=[1.0, 0.9, 0.8, 0.7]),
+    # PAPER.md Table V (L757-782, sec. V.C): 40-query sets vs a Swiss-Prot-sized DB.
+    # Homogeneous: sizes 4,500..5,000 ("range in size from 4500 to 5000", L762-763);
+    # heterogeneous: sizes 4..35,213 ("between 4 ... and 35213", L763-764).  Lengths
+    # evenly spaced over each range (sum 190k / 704k; the paper's own cells, App. D,
+    # imply sums of ~190k and ~700k against its 190.7M-residue UniProt).
+    "t5hom": dict(db_seed=2, n_db=570_000, kind=0, q_seed=6,
+                  q_lens=[4500 + (500 * i) // 39 for i in range(40)], plant_ids=[1.0, 0.8]),
+    "t5het": dict(db_seed=2, n_db=570_000, kind=0, q_seed=7,
+                  q_lens=[4 + ((35213 - 4) * i) // 39 for i in range(40)], plant_ids=[1.0, 0.8]),
 }
 
 

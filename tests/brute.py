@@ -78,3 +78,59 @@ def score_alignment(top: str, bottom: str, ma: int, mi: int, g: int) -> int:
         else:
             s += mi
     return s
+
+
+def brute_local_chains(q, d, S, gs: int, ge: int):
+    """Every optimal local alignment as its chain of aligned pairs, by the same
+    exhaustive enumeration as brute_local(): (best, [chain, ...]) with chain a
+    tuple of (i, j) pairs (0-based).  For m, n <= ~7."""
+    m, n = len(q), len(d)
+
+    def gap(k: int) -> int:
+        return gs + k * ge if k > 0 else 0
+
+    best, chains = 0, []
+    stack = [(((i, j),), int(S[q[i]][d[j]])) for i in range(m) for j in range(n)]
+    while stack:
+        ch, sc = stack.pop()
+        if sc > best:
+            best, chains = sc, [ch]
+        elif sc == best and sc > 0:
+            chains.append(ch)
+        i, j = ch[-1]
+        for i2 in range(i + 1, m):
+            gi = gap(i2 - i - 1)
+            for j2 in range(j + 1, n):
+                stack.append((ch + ((i2, j2),), sc - gi - gap(j2 - j - 1) + int(S[q[i2]][d[j2]])))
+    return best, chains
+
+
+def cigar_pairs(q_begin: int, d_begin: int, ops):
+    """Aligned (i, j) pairs of a run-length op list (op 0 = M, 1 = I, 2 = D)."""
+    i, j, out = q_begin, d_begin, []
+    for c in ops:
+        k, op = c >> 2, c & 3
+        for _ in range(k):
+            if op == 0:
+                out.append((i, j)); i += 1; j += 1
+            elif op == 1:
+                i += 1
+            else:
+                j += 1
+    return tuple(out), i - 1, j - 1
+
+
+def score_cigar(q, d, q_begin: int, d_begin: int, ops, S, gs: int, ge: int) -> int:
+    """Score of a GIVEN alignment in run-length form (sec. II.A: sum of
+    the column scores; a gap run of length k costs Gs + k*Ge, reading R-1)."""
+    i, j, s = q_begin, d_begin, 0
+    for c in ops:
+        k, op = c >> 2, c & 3
+        if op == 0:
+            for _ in range(k):
+                s += int(S[q[i]][d[j]]); i += 1; j += 1
+        elif op == 1:
+            s -= gs + k * ge; i += k
+        else:
+            s -= gs + k * ge; j += k
+    return s

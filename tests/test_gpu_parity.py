@@ -259,3 +259,24 @@ def test_query_packing(pack, thr):
         opts["overflow_threshold"] = thr
     got = gpu_scores(qc, qo, dc, do, opts=opts)
     np.testing.assert_array_equal(got, oracle_scores(qc, qo, dc, do))
+
+
+@pytest.mark.parametrize("name", ["t5hom", "t5het"])
+def test_table5_query_sets_sampled(name):
+    """PAPER.md Table V query sets (40 homogeneous 4,500-5,000 aa / heterogeneous
+    4-35,213 aa queries) against the Swiss-Prot-sized DB, on the GPU in full; the
+    oracle checks a seeded sample of DB sequences plus planted homologs and top hits."""
+    c = swgen.make_config(name)
+    got = gpu_scores(c["qcodes"], c["qoff"], c["dcodes"], c["doff"])
+    N = len(c["doff"]) - 1
+    rng = np.random.default_rng(57)
+    sample = set(rng.choice(N, size=40, replace=False).tolist())
+    sample |= {p[0] for p in c["plants"][::4]}
+    sample |= set(np.argsort(got.max(axis=0))[-5:].tolist())
+    idx = np.array(sorted(sample), dtype=np.int64)
+    lens = c["doff"][idx + 1] - c["doff"][idx]
+    sub_off = np.zeros(len(idx) + 1, dtype=np.int64)
+    np.cumsum(lens, out=sub_off[1:])
+    sub = np.concatenate([c["dcodes"][c["doff"][i]:c["doff"][i + 1]] for i in idx])
+    ref = oracle_scores(c["qcodes"], c["qoff"], sub, sub_off, procs=16)
+    np.testing.assert_array_equal(got[:, idx], ref)

@@ -18,6 +18,7 @@ import pytest
 
 import oracle
 from oracle.blosum62 import blosum62, encode
+from tests import brute
 from tests.brute import brute_local, linear_sw, score_alignment, ungapped_best
 
 GOLD = os.path.join(os.path.dirname(__file__), "golden")
@@ -190,3 +191,66 @@ def test_search_matches_pairs_and_procs():
 def test_bad_code_raises():
     with pytest.raises(ValueError):
         oracle.gotoh_score(np.array([30], np.uint8), np.array([1], np.uint8), B62, 10, 2)
+
+
+# ---------------------------------------------------------------------------
+# Alignment: end cell, start cell and path of the best local
+# alignment (oracle.gotoh_align), pinned against the exhaustive enumerator.
+
+def _rand_case(rng, mmax=7, nmax=7, alpha=5):
+    m, n = int(rng.integers(1, mmax + 1)), int(rng.integers(1, nmax + 1))
+    q = rng.integers(0, alpha, size=m).astype(np.uint8)
+    d = rng.integers(0, alpha, size=n).astype(np.uint8)
+    S = rng.integers(-4, 7, size=(alpha, alpha)).astype(np.int32)   # asymmetric on purpose
+    gs, ge = int(rng.integers(0, 6)), int(rng.integers(1, 4))
+    return q, d, S, gs, ge
+
+
+def test_align_end_and_path_vs_brute_force():
+    """Score = the brute-force optimum; end = the optimal end with the smallest j,
+    then smallest i (reading R-13); the returned path is one of the optimal
+    alignments (chain of aligned pairs) and re-scores to the score."""
+    rng = np.random.default_rng(505)
+    for _ in range(250):
+        q, d, S, gs, ge = _rand_case(rng)
+        sc, qb, qe, db, de, ops = oracle.gotoh_align(q, d, S, gs, ge)
+        best, chains = brute.brute_local_chains(q, d, S, gs, ge)
+        assert sc == best
+        if best == 0:
+            assert (qb, qe, db, de, ops) == (-1, -1, -1, -1, [])
+            continue
+        ends = sorted({(c[-1][1], c[-1][0]) for c in chains})   # (j, i)
+        assert (de, qe) == ends[0]
+        pairs, qe2, de2 = brute.cigar_pairs(qb, db, ops)
+        assert (qe2, de2) == (qe, de) and pairs[0] == (qb, db)
+        assert pairs in set(chains)
+        assert brute.score_cigar(q, d, qb, db, ops, S, gs, ge) == sc
+
+
+def test_align_rescores_on_larger_inputs():
+    """Beyond brute-force sizes: the path re-scores to the score and the score
+    equals the linear-space scorer (two independent formulations)."""
+    rng = np.random.default_rng(506)
+    S = B62
+    for _ in range(40):
+        m, n = int(rng.integers(1, 120)), int(rng.integers(1, 160))
+        q = rng.integers(0, 20, size=m).astype(np.uint8)
+        d = rng.integers(0, 20, size=n).astype(np.uint8)
+        if rng.random() < 0.5:  # plant a homologous stretch so paths have gaps
+            k = min(m, n) // 2
+            d[:k] = q[:k]
+            d[k // 2] = (d[k // 2] + 3) % 20
+        sc, qb, qe, db, de, ops = oracle.gotoh_align(q, d, S, 10, 2)
+        assert sc == oracle.gotoh_score(q, d, S, 10, 2)
+        if sc:
+            assert brute.score_cigar(q, d, qb, db, ops, S, 10, 2) == sc
+            assert ops[0] & 3 == 0 and ops[-1] & 3 == 0      # local alignments start and end on a pair
+
+
+def test_align_fig1_linear_gaps():
+    """Fig. 1 (L137-143) pair, ma +1 / mi -1 / linear g -2 (Gs = 0, Ge = 2): the
+    local optimum 5 and a path that re-scores to it."""
+    q, d, S = _dna("ACTTGTCCG"), _dna("ATTGTCAG"), _dna_matrix(1, -1)
+    sc, qb, qe, db, de, ops = oracle.gotoh_align(q, d, S, 0, 2)
+    assert sc == 5
+    assert brute.score_cigar(q, d, qb, db, ops, S, 0, 2) == 5

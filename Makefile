@@ -9,13 +9,18 @@ OBJ     := build/obj
 LIB     := $(PKG)/libswdual.so
 NVFLAGS := $(ARCH) -O3 -lineinfo -std=c++17 -Xcompiler -fPIC,-Wall -Iinclude
 HDRS    := include/swdual.h $(wildcard $(SRC)/*.h $(SRC)/*.cuh)
-OBJS    := $(OBJ)/kernels.o $(OBJ)/engine.o $(OBJ)/packer.o $(OBJ)/sched.o
+OBJS    := $(OBJ)/kernels.o $(OBJ)/align.o $(OBJ)/cpu_striped.o $(OBJ)/engine.o $(OBJ)/packer.o $(OBJ)/sched.o
 
 all: $(LIB)
 
 $(OBJ)/%.o: $(SRC)/%.cu $(HDRS)
 	@mkdir -p $(OBJ)
 	$(NVCC) $(NVFLAGS) -c $< -o $@
+
+# CPU-type PE kernel (hybrid SWDUAL): AVX2 in this file only; sw_search_cpu checks the CPU first
+$(OBJ)/cpu_striped.o: $(SRC)/cpu_striped.cpp $(HDRS)
+	@mkdir -p $(OBJ)
+	$(NVCC) $(NVFLAGS) -Xcompiler -mavx2 -c $< -o $@
 
 $(OBJ)/%.o: $(SRC)/%.cpp $(HDRS)
 	@mkdir -p $(OBJ)

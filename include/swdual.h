@@ -90,6 +90,60 @@ int32_t sw_search(sw_handle_t h, const uint8_t* q_codes, const int64_t* q_offset
                   sw_db_t db, const int8_t* matrix, int32_t gap_open, int32_t gap_extend, int32_t* scores,
                   void* cuda_stream);
 
+/*
+ * Best local alignment of selected (query, database sequence) pairs -- its
+ * score, end cell, start cell and path (every
+ * matrix element "keeps the cell that was used to produce the value", followed
+ * back from the maximal cell).  Typical use: the top hits of an sw_search.
+ *   q_codes, q_offsets, n_queries   host, queries as for sw_search.
+ *   db          a DB loaded on this handle.
+ *   pairs       host, int32[n_pairs][2] = (query index, DB sequence index in the
+ *               caller's order).
+ *   matrix, gap_open, gap_extend    as for sw_search.
+ *   out5        host, int32[n_pairs][5] = {score, q_begin, q_end, d_begin, d_end}:
+ *               0-based inclusive residue ranges of the alignment; all four -1
+ *               when the score is 0 (no alignment).
+ *   ops         host, uint32 run-length operations (len << 2 | op), op 0 = M
+ *               (aligned pair), 1 = I (query residue vs gap), 2 = D (DB residue vs
+ *               gap), start to end; pair k uses ops[ops_offsets[k] ..
+ *               ops_offsets[k+1]) and n_ops[k] (host, int32[n_pairs]) receives
+ *               the count.  A region of m_q + n_d entries always suffices.
+ *   ops_offsets host, int64[n_pairs + 1], non-decreasing.
+ * Tie-breaks (R-13): end cell = maximal H with the smallest DB position,
+ * then the smallest query position; traceback prefers the diagonal, then E
+ * (gap in the query), then F; a gap is opened rather than extended on a tie.
+ * Synchronous: returns after the results are in the host buffers.
+ * Scores are exact int32 (no int16 path).  Work: int32 wavefront kernel with a
+ * 4-bit traceback code per cell kept in device memory (m*n/2 bytes per pair,
+ * batched under the "align_workspace_mb" option), then one thread per pair
+ * walks it.
+ * Errors: SW_EINVAL (bad index, code, gaps, null pointer, a region too small
+ * for the path), SW_ESTATE, SW_ENOMEM, SW_ECUDA, SW_EUNSUPPORTED (a sequence
+ * longer than 2^20 - 64).
+ */
+int32_t sw_align(sw_handle_t h, const uint8_t* q_codes, const int64_t* q_offsets, int32_t n_queries, sw_db_t db,
+                 const int32_t* pairs, int32_t n_pairs, const int8_t* matrix, int32_t gap_open, int32_t gap_extend,
+                 int32_t* out5, uint32_t* ops, const int64_t* ops_offsets, int32_t* n_ops, void* cuda_stream);
+
+/*
+ * CPU-type processing element of the hybrid SWDUAL (PAPER.md
+ * sec. III: tasks are placed on "m CPUs and k GPUs" by the dual
+ * approximation, sw_schedule_dual).  Host-only, no handle, no GPU: scores
+ * n_queries x n_seqs pairs on n_threads host threads with a striped AVX2 int16
+ * kernel (saturation-flagged pairs re-scored in int32) -- the work the paper's
+ * CPU workers do (L529-539).  This is a scheduling target the caller chooses
+ * for some tasks, never a fallback of sw_search.
+ *   q_codes, q_offsets, n_queries   host, as for sw_search.
+ *   db_codes, db_offsets, n_seqs    host, as for sw_load_db (not packed).
+ *   alphabet_size, matrix, gap_open, gap_extend   as for sw_load_db / sw_search.
+ *   n_threads   >= 1.
+ *   scores      host, int32[n_queries][n_seqs].
+ * Synchronous.  Errors: SW_EINVAL (as sw_search), SW_EUNSUPPORTED (no AVX2).
+ */
+int32_t sw_search_cpu(const uint8_t* q_codes, const int64_t* q_offsets, int32_t n_queries, const uint8_t* db_codes,
+                      const int64_t* db_offsets, int64_t n_seqs, int32_t alphabet_size, const int8_t* matrix,
+                      int32_t gap_open, int32_t gap_extend, int32_t n_threads, int32_t* scores);
+
 int32_t sw_free_db(sw_db_t db);
 int32_t sw_free(sw_handle_t h); /* frees the handle and any DBs still attached */
 
@@ -138,11 +192,24 @@ int32_t sw_last_stats(sw_handle_t h, sw_stats_t* out);
  *   "timing_accumulate"   1: short_ms/long_ms of sw_last_stats sum every search
  *                         since the last "timing_reset" (0: the last search only)
  *   "timing_reset"        clear the accumulated kernel events
+ *   "align_workspace_mb"  device memory for sw_align's traceback codes per batch
+ *                         (default 2048; a pair needing more runs alone)
  */
 int32_t sw_set_option(sw_handle_t h, const char* key, int64_t value);
 
 /* ASCII -> NCBI protein codes "ARNDCQEGHILKMFPSTWYVBZX*" (lower case folded, unknown -> X). */
 int32_t sw_encode_ascii(const char* s, int64_t n, uint8_t* out);
+
+/*
+ * ASCII -> nucleotide codes (DNA over
+ * {A, T, G, C}, RNA over {A, U, G, C}): A 0, C 1, G 2, T and U 3, anything else
+ * (N, IUPAC ambiguity letters) 4; lower case folded.  Alphabet size 5: load the
+ * DB with alphabet_size = 5 and score with a 5 x 5 match/mismatch matrix (the
+ * paper's ma / mi, L127-133; the Python binding's nucleotide_matrix); the
+ * linear gap g of Eq. (1) (L159-165) is gap_open = 0, gap_extend = -g.
+ * s, out host; out may alias s.  Errors: SW_EINVAL (n < 0, NULL with n > 0).
+ */
+int32_t sw_encode_nucleotide(const char* s, int64_t n, uint8_t* out);
 
 /*
  * Dual-approximation placement (sec. III): n_tasks tasks,

@@ -80,6 +80,7 @@ class Handle:
         check(lib().sw_load_db(self.ptr, _vp(codes) if codes.size else None, _vp(offsets), n, int(alphabet_size),
                                _stream_ptr(stream), ctypes.byref(out)), self.ptr)
         db = Database(self, out, n)
+        db.seq_lens = np.diff(offsets)
         self._dbs.append(db)
         return db
 
@@ -111,6 +112,41 @@ class Handle:
                               _vp(matrix), int(gap_open), int(gap_extend), optr, _stream_ptr(stream)), self.ptr)
         return out
 
+    def align(self, q_codes, q_offsets, db: Database, pairs, matrix, gap_open: int = 10, gap_extend: int = 2,
+              stream=None):
+        """sw_align: best local alignment of each (query index, DB index) pair.
+
+        Returns a list of (score, q_begin, q_end, d_begin, d_end, ops), ops the
+        run-length operations (len << 2 | op; op 0 = M, 1 = I, 2 = D), start to end.
+        """
+        q_codes = _host(q_codes, np.uint8)
+        q_offsets = _host(q_offsets, np.int64)
+        matrix = _host(matrix, np.int8)
+        pairs = _host(pairs, np.int32).reshape(-1, 2)
+        nq = len(q_offsets) - 1
+        n = len(pairs)
+        if n == 0:
+            return []
+        info_lens = self._seq_lens(db)
+        qlens = np.diff(q_offsets)
+        caps = qlens[pairs[:, 0].clip(0, max(nq - 1, 0))] + info_lens[pairs[:, 1].clip(0, len(info_lens) - 1)]
+        offs = np.zeros(n + 1, dtype=np.int64)
+        np.cumsum(caps, out=offs[1:])
+        ops = np.zeros(max(int(offs[-1]), 1), dtype=np.uint32)
+        out5 = np.zeros((n, 5), dtype=np.int32)
+        nops = np.zeros(n, dtype=np.int32)
+        check(lib().sw_align(self.ptr, _vp(q_codes) if q_codes.size else None, _vp(q_offsets), nq, db.ptr,
+                             _vp(pairs), n, _vp(matrix), int(gap_open), int(gap_extend), _vp(out5), _vp(ops),
+                             _vp(offs), _vp(nops), _stream_ptr(stream)), self.ptr)
+        return [tuple(int(x) for x in out5[k]) + ([int(x) for x in ops[offs[k]:offs[k] + nops[k]]],)
+                for k in range(n)]
+
+    def _seq_lens(self, db: Database) -> np.ndarray:
+        lens = getattr(db, "seq_lens", None)
+        if lens is None:
+            raise ValueError("align: load the DB through Handle.load_db (sequence lengths needed)")
+        return lens
+
     def last_stats(self) -> dict:
         s = Stats()
         check(lib().sw_last_stats(self.ptr, ctypes.byref(s)), self.ptr)
@@ -141,6 +177,33 @@ def encode_ascii(s: str) -> np.ndarray:
     b = s.encode("ascii", "replace")
     out = np.zeros(len(b), dtype=np.uint8)
     check(lib().sw_encode_ascii(b, len(b), _vp(out) if len(b) else None))
+    return out
+
+
+def search_cpu(q_codes, q_offsets, db_codes, db_offsets, matrix, gap_open: int = 10, gap_extend: int = 2,
+               alphabet_size: int = 24, n_threads: int = 1) -> np.ndarray:
+    """sw_search_cpu: a CPU-type PE of the hybrid SWDUAL (host AVX2 kernel), int32[Q, N].
+
+    A scheduling target for tasks the dual approximation places on CPUs, not a
+    fallback of Handle.search (which never routes here)."""
+    q_codes = _host(q_codes, np.uint8)
+    q_offsets = _host(q_offsets, np.int64)
+    db_codes = _host(db_codes, np.uint8)
+    db_offsets = _host(db_offsets, np.int64)
+    matrix = _host(matrix, np.int8)
+    nq, n = len(q_offsets) - 1, len(db_offsets) - 1
+    out = np.zeros((nq, n), dtype=np.int32)
+    check(lib().sw_search_cpu(_vp(q_codes) if q_codes.size else None, _vp(q_offsets), nq,
+                              _vp(db_codes) if db_codes.size else None, _vp(db_offsets), n, int(alphabet_size),
+                              _vp(matrix), int(gap_open), int(gap_extend), int(n_threads), _vp(out) if out.size else None))
+    return out
+
+
+def encode_nucleotide(s: str) -> np.ndarray:
+    """sw_encode_nucleotide: DNA/RNA string -> codes A 0, C 1, G 2, T/U 3, other 4."""
+    b = s.encode("ascii", "replace")
+    out = np.zeros(len(b), dtype=np.uint8)
+    check(lib().sw_encode_nucleotide(b, len(b), _vp(out) if len(b) else None))
     return out
 
 

@@ -51,3 +51,16 @@ def blosum62() -> np.ndarray:
         for j, v in enumerate(vals):
             M[i, j] = M[j, i] = v
     return M
+
+
+NUCLEOTIDES = "ACGTN"  # sw_encode_nucleotide codes 0..4 (U shares T's code)
+
+
+def nucleotide_matrix(match: int = 1, mismatch: int = -1, n_score: int = None) -> np.ndarray:
+    """5 x 5 int8 match/mismatch matrix over ACGTN (ma for
+    identical bases, mi otherwise; Fig. 1 uses ma = +1, mi = -1).  N scores
+    n_score against everything (default: mismatch)."""
+    M = np.full((5, 5), mismatch, dtype=np.int8)
+    np.fill_diagonal(M, match)
+    M[4, :] = M[:, 4] = mismatch if n_score is None else n_score
+    return M

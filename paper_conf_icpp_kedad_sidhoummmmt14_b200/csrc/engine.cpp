@@ -12,6 +12,7 @@
 #include <algorithm>
 #include <atomic>
 #include <cstdio>
+#include <cstdlib>
 #include <cstring>
 #include <mutex>
 #include <new>
@@ -107,6 +108,9 @@ struct sw_handle_s {
   int64_t opt_pack_queries = 1; // mode-1 slots: fill the shorter half with further queries (strip-aligned)
   int64_t opt_bank_copy = 1;    // query-pair profile: second smem copy shifted by 64 B for odd lane groups
   int64_t opt_pack_long = 0;    // 1: several long pairs per CTA item when a query has fewer strips than warps
+  int64_t opt_align_ws_mb = 2048;  // sw_align: traceback-code workspace per batch
+  // sw_align scratch (separate from sw_search's: a search may still be running on another stream)
+  DevBuf a_qcodes, a_qoff, a_matrix, a_items, a_links, a_trace, a_best, a_ops, a_out, a_counter;
   // last-search bookkeeping
   sw_stats_t stats{};
   cudaStream_t last_stream = nullptr;
@@ -130,6 +134,7 @@ struct sw_db_s {
   std::vector<int64_t> len_prefix;  // [np+1] prefix of padded pair lengths
   DevBuf dlofs;
   DevBuf stream, dpairs;
+  std::vector<int64_t> seq_loc;  // caller index -> 2 * pair + half (-1: empty); built on first sw_align
 };
 
 static int32_t set_err(sw_handle_s* h, int32_t code, const std::string& m) {
@@ -245,6 +250,9 @@ int32_t sw_set_option(sw_handle_t h, const char* key, int64_t value) {
   } else if (k == "t_long") {
     if (value < 0) return set_err(h, SW_EINVAL, "t_long must be >= 0");
     h->opt_t_long = value;
+  } else if (k == "align_workspace_mb") {
+    if (value < 1) return set_err(h, SW_EINVAL, "sw_set_option: align_workspace_mb must be >= 1");
+    h->opt_align_ws_mb = value;
   } else if (k == "pack_long") {
     h->opt_pack_long = value;
   } else if (k == "pack_queries") {
@@ -918,6 +926,158 @@ int32_t sw_search(sw_handle_t h, const uint8_t* q_codes, const int64_t* q_offset
   });
 }
 
+// ----------------------------------------------------------------------------
+// sw_align: int32 wavefront with 4-bit traceback codes, then a
+// per-pair walk (align.cu).  Pairs are batched so that the codes of a batch fit
+// the workspace budget.
+int32_t sw_align(sw_handle_t h, const uint8_t* q_codes, const int64_t* q_offsets, int32_t n_queries, sw_db_t db,
+                 const int32_t* pairs, int32_t n_pairs, const int8_t* matrix, int32_t gap_open, int32_t gap_extend,
+                 int32_t* out5, uint32_t* ops, const int64_t* ops_offsets, int32_t* n_ops, void* cuda_stream) {
+  if (!h) return set_err(nullptr, SW_EINVAL, "sw_align: handle is NULL");
+  return guarded(h, [&] {
+    if (!db) fail(SW_EINVAL, "sw_align: db is NULL");
+    if (db->h != h) fail(SW_ESTATE, "sw_align: db belongs to another handle");
+    if (n_pairs < 0 || n_queries < 0) fail(SW_EINVAL, "sw_align: negative count");
+    if (n_pairs == 0) return;
+    if (!pairs || !out5 || !n_ops || !ops_offsets || !q_offsets || !matrix)
+      fail(SW_EINVAL, "sw_align: NULL argument");
+    if (gap_open < 0 || gap_extend < 0) fail(SW_EINVAL, "sw_align: gap penalties must be >= 0");
+    if (int64_t(gap_open) + gap_extend > (int64_t(1) << 24)) fail(SW_EINVAL, "sw_align: gap penalties too large");
+    const int alpha = db->alpha;
+    SW_CK(cudaSetDevice(h->device));
+    cudaStream_t st = reinterpret_cast<cudaStream_t>(cuda_stream);
+    std::vector<int64_t> qlen(static_cast<size_t>(n_queries));
+    int64_t qtot = 0;
+    for (int i = 0; i < n_queries; ++i) {
+      qlen[size_t(i)] = q_offsets[i + 1] - q_offsets[i];
+      if (qlen[size_t(i)] < 0) fail(SW_EINVAL, "sw_align: q_offsets not non-decreasing");
+      if (qlen[size_t(i)] > (int64_t(1) << 30)) fail(SW_EUNSUPPORTED, "sw_align: query longer than 2^30");
+      qtot += qlen[size_t(i)];
+    }
+    if (qtot > 0 && !q_codes) fail(SW_EINVAL, "sw_align: q_codes is NULL");
+    const uint8_t* qbase = q_codes ? q_codes + q_offsets[0] : nullptr;
+    for (int64_t i = 0; i < qtot; ++i)
+      if (qbase[i] >= alpha) fail(SW_EINVAL, "sw_align: query code >= alphabet_size");
+    if (db->seq_loc.empty()) {
+      db->seq_loc.assign(size_t(db->n_seqs), -1);
+      for (size_t p = 0; p < db->pairs.size(); ++p) {
+        db->seq_loc[size_t(db->pairs[p].id0)] = int64_t(2 * p);
+        if (db->pairs[p].id1 >= 0) db->seq_loc[size_t(db->pairs[p].id1)] = int64_t(2 * p + 1);
+      }
+    }
+    // items (pairs with an empty side are answered on the host)
+    std::vector<AlignItem> items;
+    std::vector<int32_t> item_pair;  // caller index of each item
+    std::vector<int64_t> words;      // trace words per item
+    for (int32_t k = 0; k < n_pairs; ++k) {
+      const int32_t q = pairs[2 * k], d = pairs[2 * k + 1];
+      if (q < 0 || q >= n_queries) fail(SW_EINVAL, "sw_align: query index out of range");
+      if (d < 0 || int64_t(d) >= db->n_seqs) fail(SW_EINVAL, "sw_align: DB index out of range");
+      if (ops_offsets[k + 1] < ops_offsets[k]) fail(SW_EINVAL, "sw_align: ops_offsets not non-decreasing");
+      const int64_t m = qlen[size_t(q)], n = db->seq_len[size_t(d)];
+      n_ops[k] = 0;
+      out5[5 * k] = 0;
+      for (int c = 1; c < 5; ++c) out5[5 * k + c] = -1;
+      if (m == 0 || n == 0) continue;
+      if (n > (int64_t(1) << 20) - 64) fail(SW_EUNSUPPORTED, "sw_align: DB sequence longer than 2^20 - 64");
+      if (!ops && ops_offsets[k + 1] > ops_offsets[k]) fail(SW_EINVAL, "sw_align: ops is NULL");
+      AlignItem it{};
+      it.q = q;
+      it.pair = int32_t(db->seq_loc[size_t(d)] >> 1);
+      it.half = int32_t(db->seq_loc[size_t(d)] & 1);
+      it.n = int32_t(n);
+      it.ops_cap = int32_t(std::min<int64_t>(ops_offsets[k + 1] - ops_offsets[k], m + n + 1));
+      items.push_back(it);
+      item_pair.push_back(k);
+      words.push_back((m + 255) / 256 * (((n + 3) & ~int64_t(3)) + 32) * 32);
+    }
+    if (items.empty()) return;
+    // device inputs
+    SW_CK(h->a_qcodes.ensure(size_t(std::max<int64_t>(qtot, 1))));
+    SW_CK(h->a_qoff.ensure(size_t(n_queries + 1) * sizeof(int64_t)));
+    SW_CK(h->a_matrix.ensure(size_t(alpha * alpha)));
+    std::vector<int64_t> qoff0(static_cast<size_t>(n_queries + 1));
+    for (int i = 0; i <= n_queries; ++i) qoff0[size_t(i)] = q_offsets[i] - q_offsets[0];
+    if (qtot) SW_CK(cudaMemcpyAsync(h->a_qcodes.p, qbase, size_t(qtot), cudaMemcpyHostToDevice, st));
+    SW_CK(cudaMemcpyAsync(h->a_qoff.p, qoff0.data(), qoff0.size() * sizeof(int64_t), cudaMemcpyHostToDevice, st));
+    SW_CK(cudaMemcpyAsync(h->a_matrix.p, matrix, size_t(alpha * alpha), cudaMemcpyHostToDevice, st));
+    SW_CK(h->a_counter.ensure(sizeof(int)));
+    const int64_t budget = h->opt_align_ws_mb * (int64_t(1) << 20) / 4;  // words
+    std::vector<uint32_t> hops;
+    std::vector<int32_t> hout;
+    size_t b0 = 0;
+    while (b0 < items.size()) {
+      // batch [b0, b1): trace words within budget (at least one item)
+      size_t b1 = b0;
+      int64_t tw = 0, ow = 0;
+      int bcap = 0;
+      while (b1 < items.size() && (b1 == b0 || tw + words[b1] <= budget)) {
+        items[b1].trace_off = tw;
+        items[b1].ops_off = ow;
+        tw += words[b1];
+        ow += items[b1].ops_cap;
+        bcap = std::max(bcap, ((items[b1].n + 3) & ~3) + 32 + 8);
+        ++b1;
+      }
+      const int nb = int(b1 - b0);
+      SW_CK(h->a_items.ensure(size_t(nb) * sizeof(AlignItem)));
+      SW_CK(h->a_trace.ensure(size_t(tw) * sizeof(uint32_t)));
+      SW_CK(h->a_best.ensure(size_t(nb) * sizeof(int4)));
+      SW_CK(h->a_ops.ensure(size_t(std::max<int64_t>(ow, 1)) * sizeof(uint32_t)));
+      SW_CK(h->a_out.ensure(size_t(nb) * 6 * sizeof(int32_t)));
+      int grid = std::min(nb, h->sms * 4);
+      const int64_t link_budget = int64_t(256) << 20;  // bytes of warp link rows
+      const int64_t per_cta = int64_t(ALIGN_WARPS) * bcap * int64_t(sizeof(int2));
+      grid = int(std::max<int64_t>(1, std::min<int64_t>(grid, std::max<int64_t>(h->sms, link_budget / per_cta))));
+      SW_CK(h->a_links.ensure(size_t(grid) * size_t(per_cta)));
+      SW_CK(cudaMemcpyAsync(h->a_items.p, items.data() + b0, size_t(nb) * sizeof(AlignItem), cudaMemcpyHostToDevice,
+                            st));
+      SW_CK(cudaMemsetAsync(h->a_counter.p, 0, sizeof(int), st));
+      AlignArgs a{};
+      a.qcodes = h->a_qcodes.as<uint8_t>();
+      a.qoff = h->a_qoff.as<int64_t>();
+      a.stream = db->stream.as<uint16_t>();
+      a.pairs = db->dpairs.as<PairRec>();
+      a.matrix = h->a_matrix.as<int8_t>();
+      a.alpha = alpha;
+      a.items = h->a_items.as<AlignItem>();
+      a.n_items = nb;
+      a.work_counter = h->a_counter.as<int>();
+      a.links = h->a_links.as<int2>();
+      a.bcap = bcap;
+      a.trace = h->a_trace.as<uint32_t>();
+      a.best = h->a_best.as<int4>();
+      a.ops = h->a_ops.as<uint32_t>();
+      a.out = h->a_out.as<int32_t>();
+      a.Gs = gap_open;
+      a.Ge = gap_extend;
+      SW_CK(launch_align(grid, a, st));
+      hout.resize(size_t(nb) * 6);
+      hops.resize(size_t(std::max<int64_t>(ow, 1)));
+      SW_CK(cudaMemcpyAsync(hout.data(), h->a_out.p, hout.size() * sizeof(int32_t), cudaMemcpyDeviceToHost, st));
+      if (ow) SW_CK(cudaMemcpyAsync(hops.data(), h->a_ops.p, size_t(ow) * sizeof(uint32_t), cudaMemcpyDeviceToHost, st));
+      SW_CK(cudaStreamSynchronize(st));
+      if (const char* dump = std::getenv("SWDUAL_ALIGN_DUMP")) {  // debugging aid: raw traceback codes
+        std::vector<uint32_t> tr(static_cast<size_t>(tw));
+        SW_CK(cudaMemcpy(tr.data(), h->a_trace.p, size_t(tw) * 4, cudaMemcpyDeviceToHost));
+        if (FILE* f = std::fopen(dump, "wb")) { std::fwrite(tr.data(), 4, tr.size(), f); std::fclose(f); }
+      }
+      for (int x = 0; x < nb; ++x) {
+        const AlignItem& it = items[b0 + size_t(x)];
+        const int32_t k = item_pair[b0 + size_t(x)];
+        const int32_t* o = &hout[size_t(x) * 6];
+        if (o[5] < 0 || o[5] > ops_offsets[k + 1] - ops_offsets[k])
+          fail(SW_EINVAL, "sw_align: ops region of pair " + std::to_string(k) + " too small (needs " +
+                              std::to_string(o[5] < 0 ? -o[5] : o[5]) + " entries)");
+        for (int c = 0; c < 5; ++c) out5[5 * k + c] = o[c];
+        n_ops[k] = o[5];
+        if (o[5]) std::memcpy(ops + ops_offsets[k], &hops[size_t(it.ops_off)], size_t(o[5]) * sizeof(uint32_t));
+      }
+      b0 = b1;
+    }
+  });
+}
+
 int32_t sw_last_stats(sw_handle_t h, sw_stats_t* out) {
   if (!h || !out) return set_err(h, SW_EINVAL, "sw_last_stats: NULL argument");
   return guarded(h, [&] {
@@ -992,6 +1152,47 @@ int32_t sw_encode_ascii(const char* s, int64_t n, uint8_t* out) {
   }
   lut[uint8_t('U')] = lut[uint8_t('u')] = 4;   // selenocysteine -> C
   lut[uint8_t('O')] = lut[uint8_t('o')] = 11;  // pyrrolysine -> K
+  for (int64_t i = 0; i < n; ++i) out[i] = lut[uint8_t(s[i])];
+  return SW_OK;
+}
+
+int32_t sw_search_cpu(const uint8_t* q_codes, const int64_t* q_offsets, int32_t n_queries, const uint8_t* db_codes,
+                      const int64_t* db_offsets, int64_t n_seqs, int32_t alphabet_size, const int8_t* matrix,
+                      int32_t gap_open, int32_t gap_extend, int32_t n_threads, int32_t* scores) {
+  return guarded(nullptr, [&] {
+    if (n_queries < 0 || n_seqs < 0) fail(SW_EINVAL, "sw_search_cpu: negative count");
+    if (alphabet_size < 1 || alphabet_size > 32) fail(SW_EINVAL, "sw_search_cpu: alphabet_size must be 1..32");
+    if (gap_open < 0 || gap_extend < 0) fail(SW_EINVAL, "sw_search_cpu: gap penalties must be >= 0");
+    if (int64_t(gap_open) + gap_extend > 32767) fail(SW_EINVAL, "sw_search_cpu: gap_open + gap_extend > 32767");
+    if (n_threads < 1) fail(SW_EINVAL, "sw_search_cpu: n_threads must be >= 1");
+    if (n_queries == 0 || n_seqs == 0) return;
+    if (!q_offsets || !db_offsets || !matrix || !scores) fail(SW_EINVAL, "sw_search_cpu: NULL argument");
+    if (!__builtin_cpu_supports("avx2")) fail(SW_EUNSUPPORTED, "sw_search_cpu: the host CPU has no AVX2");
+    auto check_codes = [&](const uint8_t* c, const int64_t* off, int64_t n, const char* what) {
+      for (int64_t i = 0; i < n; ++i)
+        if (off[i + 1] < off[i]) fail(SW_EINVAL, std::string("sw_search_cpu: ") + what + " offsets not non-decreasing");
+      const int64_t tot = off[n] - off[0];
+      if (tot > 0 && !c) fail(SW_EINVAL, std::string("sw_search_cpu: ") + what + " codes NULL");
+      for (int64_t i = 0; i < tot; ++i)
+        if (c[i] >= alphabet_size) fail(SW_EINVAL, std::string("sw_search_cpu: ") + what + " code >= alphabet_size");
+    };
+    check_codes(q_codes, q_offsets, n_queries, "query");
+    check_codes(db_codes, db_offsets, n_seqs, "DB");
+    swdual::cpu_search_avx2(q_codes, q_offsets, n_queries, db_codes, db_offsets, n_seqs, alphabet_size, matrix,
+                            gap_open, gap_extend, n_threads, scores);
+  });
+}
+
+int32_t sw_encode_nucleotide(const char* s, int64_t n, uint8_t* out) {
+  if (n < 0 || (n > 0 && (!s || !out))) return set_err(nullptr, SW_EINVAL, "sw_encode_nucleotide: bad argument");
+  uint8_t lut[256];
+  std::memset(lut, 4, sizeof(lut));  // N and every other letter
+  const char* AL = "ACGT";
+  for (int k = 0; k < 4; ++k) {
+    lut[uint8_t(AL[k])] = uint8_t(k);
+    lut[uint8_t(AL[k] - 'A' + 'a')] = uint8_t(k);
+  }
+  lut[uint8_t('U')] = lut[uint8_t('u')] = 3;  // RNA uracil pairs like T
   for (int64_t i = 0; i < n; ++i) out[i] = lut[uint8_t(s[i])];
   return SW_OK;
 }

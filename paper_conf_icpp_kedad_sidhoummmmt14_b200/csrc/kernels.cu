@@ -22,7 +22,6 @@
 
 namespace swdual {
 
-constexpr uint32_t FULL = 0xffffffffu;
 constexpr int8_t PAD_SCORE = -64;  // S[.][PAD] = S[PAD][.] <= 0 (reading R-12)
 // Intra-task mode: a strip starts consuming the row above only once its
 // producer is this many columns ahead, so producer and consumer warps of a
@@ -118,54 +117,6 @@ cudaError_t launch_build_profile_q2(const uint8_t* qa, int ma, const uint8_t* qb
   build_profile_q2_kernel<<<grid, 256, 0, st>>>(qa, ma, qb, mb, matrix, alpha, G, R, LB2, LS2, n_strips, SB2,
                                                 reinterpret_cast<uint32_t*>(prof));
   return cudaGetLastError();
-}
-
-// Progress counters of chained strips.  Within a CTA they live in shared memory
-// (CTA-scope release/acquire); between the CTAs that hold consecutive
-// "superstrips" of one long pair they live in global memory (GPU scope).
-__device__ __forceinline__ int ld_acquire_cta(const int* p) {
-  int v;
-  asm volatile("ld.acquire.cta.shared.b32 %0, [%1];"
-               : "=r"(v) : "r"(static_cast<uint32_t>(__cvta_generic_to_shared(const_cast<int*>(p)))) : "memory");
-  return v;
-}
-__device__ __forceinline__ void st_release_cta(int* p, int v) {
-  asm volatile("st.release.cta.shared.b32 [%0], %1;"
-               :: "r"(static_cast<uint32_t>(__cvta_generic_to_shared(p))), "r"(v) : "memory");
-}
-__device__ __forceinline__ int ld_acquire_gpu(const int* p) {
-  int v;
-  asm volatile("ld.acquire.gpu.global.b32 %0, [%1];" : "=r"(v) : "l"(p) : "memory");
-  return v;
-}
-__device__ __forceinline__ void st_release_gpu(int* p, int v) {
-  asm volatile("st.release.gpu.global.b32 [%0], %1;" :: "l"(p), "r"(v) : "memory");
-}
-
-// Link of a chained strip: the row above (read by lane 0) and this strip's
-// bottom row (written by the last lane), each with a progress counter.
-struct Link {
-  int* in;        // counter of the producer of the row above (nullptr: none)
-  int in_base;    // value the producer publishes before its first cell
-  bool in_gpu;    // counter in global memory (other CTA)
-  int* out;       // this strip's counter (nullptr: nobody consumes it)
-  int out_base;
-  bool out_gpu;
-};
-
-// Warp-uniform wait until a progress counter reaches `need` (one lane polls,
-// the result is broadcast, so the warp stays converged and the shuffles that
-// follow stay on the fast path).  `seen` caches the last value observed.
-__device__ __forceinline__ void wait_progress(const Link& lk, int need, int& seen) {
-  if (seen >= need) return;
-  for (;;) {
-    int v = 0;
-    if ((threadIdx.x & 31) == 0) v = lk.in_gpu ? ld_acquire_gpu(lk.in) : ld_acquire_cta(lk.in);
-    v = __shfl_sync(FULL, v, 0);
-    if (v >= need) { seen = v; break; }
-    __nanosleep(lk.in_gpu ? 256 : 64);
-  }
-  if (lk.in_gpu) __threadfence();  // lane 0 acquired; make the row visible to its later loads
 }
 
 // ---------------------------------------------------------------------------

@@ -182,4 +182,47 @@ cudaError_t launch_rescore(int grid, const RescoreArgs& a, cudaStream_t st);
 constexpr int RESCORE_WARPS = 8;
 constexpr int RESCORE_R = 8;
 
+
+// Best local alignment of selected pairs (align.cu).  One item =
+// one (query, DB sequence) pair; its traceback codes live at trace + trace_off:
+// [strip][step t][lane] u32 words, 8 rows x 4 bits per word (see align.cu).
+struct AlignItem {
+  int64_t trace_off;         // u32 words
+  int64_t ops_off;           // u32 run-length codes: this item's output region
+  int32_t q;                 // query index (qoff)
+  int32_t pair;              // packed pair holding the DB sequence
+  int32_t half;              // 0 = low byte (id0), 1 = high byte (id1)
+  int32_t n;                 // real DB sequence length
+  int32_t ops_cap;           // capacity of the output region
+  int32_t pad_;
+};
+
+struct AlignArgs {
+  const uint8_t* qcodes;     // all queries, concatenated
+  const int64_t* qoff;       // [nq+1]
+  const uint16_t* stream;
+  const PairRec* pairs;
+  const int8_t* matrix;      // alpha x alpha
+  int alpha;
+  const AlignItem* items;    // this batch
+  int n_items;
+  int* work_counter;         // zeroed
+  int2* links;               // per-CTA warp link rows, [gridDim][ALIGN_WARPS][bcap]
+  int bcap;
+  uint32_t* trace;           // traceback codes of the batch
+  int4* best;                // per item: {score, end row i (1-based), end column j (1-based), 0}
+  uint32_t* ops;             // run-length codes, per item at ops_off (written reversed, then flipped)
+  int32_t* out;              // per item: {score, q_begin, q_end, d_begin, d_end, n_ops (< 0: region too small)}
+  int32_t Gs, Ge;
+};
+
+// CPU-type PE (cpu_striped.cpp, AVX2): scores[q][d] for all pairs, host only.
+void cpu_search_avx2(const uint8_t* qcodes, const int64_t* qoff, int32_t nq, const uint8_t* dcodes,
+                     const int64_t* doff, int64_t n_seqs, int alpha, const int8_t* S, int32_t Gs, int32_t Ge,
+                     int32_t n_threads, int32_t* scores);
+
+constexpr int ALIGN_WARPS = 8;
+constexpr int ALIGN_R = 8;   // rows per lane = codes per trace word
+cudaError_t launch_align(int grid, const AlignArgs& a, cudaStream_t st);
+
 }  // namespace swdual

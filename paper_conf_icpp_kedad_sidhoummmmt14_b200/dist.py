@@ -149,3 +149,111 @@ def run(plan: Plan, rank: int, n_queries: int, n_seqs: int, score_block, dist=No
         g = gathered.cpu().numpy().reshape(world, -1)
         flats = [g[r] for r in range(world)]
     return assemble(plan, n_queries, n_seqs, flats)
+
+
+# ---------------------------------------------------------------------------
+# Hybrid SWDUAL on one box: the paper's setting of "m CPUs and
+# k GPUs" with host cores as CPU-type PEs.  Every task
+# (query, shard) has a CPU time and a GPU time from calibrated cell rates; the
+# dual approximation (sw_schedule_dual) places it; the GPU tasks run through
+# sw_search while the CPU PEs run theirs concurrently through sw_search_cpu
+# (one host thread per PE).  Opt-in: plain searches never touch the CPU path.
+
+@dataclass
+class HybridPlan:
+    shards: list[np.ndarray]
+    tasks: list[tuple[int, int]]             # (query, shard)
+    pe: np.ndarray                           # task -> PE (0..n_cpus-1 CPUs, then GPUs)
+    n_cpus: int
+    n_gpus: int
+    makespan: float
+    lam: float
+    p_cpu: np.ndarray
+    p_gpu: np.ndarray
+
+    def cpu_tasks(self, c: int):
+        return [t for t, p in zip(self.tasks, self.pe) if p == c]
+
+    def gpu_tasks(self, g: int = 0):
+        return [t for t, p in zip(self.tasks, self.pe) if p == self.n_cpus + g]
+
+
+def place_hybrid(q_lens, shards, n_cpus: int, n_gpus: int, gpu_rate: float, cpu_rate: float,
+                 shard_residues=None) -> HybridPlan:
+    """Tasks (query, shard) with p = cells / rate on each PE type (reading S-1/S-2),
+    placed by the dual approximation on n_cpus CPU PEs + n_gpus GPUs."""
+    if shard_residues is None:
+        raise ValueError("shard_residues required")
+    tasks = [(q, s) for q in range(len(q_lens)) for s in range(len(shards))]
+    cells = np.array([float(q_lens[q]) * float(shard_residues[s]) for q, s in tasks], dtype=np.float64)
+    p_cpu, p_gpu = cells / float(cpu_rate), cells / float(gpu_rate)
+    if tasks:
+        pe, mk, lam = schedule_dual(p_cpu, p_gpu, n_cpus, n_gpus)
+    else:
+        pe, mk, lam = np.zeros(0, np.int32), 0.0, 0.0
+    return HybridPlan(shards, tasks, np.asarray(pe, np.int64), n_cpus, n_gpus, mk, lam, p_cpu, p_gpu)
+
+
+class HybridDB:
+    """A database cut into shards, resident both on the GPU (one sw_db per shard,
+    loaded once) and on the host (for the CPU PEs)."""
+
+    def __init__(self, handle, db_codes, db_offsets, n_shards: int = 8, alphabet_size: int = 24):
+        self.handle = handle
+        self.alphabet_size = alphabet_size
+        self.db_offsets = np.ascontiguousarray(db_offsets, dtype=np.int64)
+        self.n_seqs = len(self.db_offsets) - 1
+        self.shards = shard_cut(self.db_offsets, n_shards)
+        self.host = [subset(db_codes, self.db_offsets, idx) for idx in self.shards]
+        self.gpu = [handle.load_db(c, o, alphabet_size=alphabet_size) for c, o in self.host]
+        self.residues = [float(o[-1] - o[0]) for _, o in self.host]
+
+    def plan(self, q_lens, n_cpus: int, gpu_rate: float, cpu_rate: float) -> HybridPlan:
+        return place_hybrid(q_lens, self.shards, n_cpus, 1, gpu_rate, cpu_rate, shard_residues=self.residues)
+
+    def search(self, q_codes, q_offsets, matrix, gap_open=10, gap_extend=2, n_cpus: int = 4,
+               gpu_rate: float = 6.5e12, cpu_rate: float = 3.0e9, plan: HybridPlan | None = None):
+        """scores int32[Q, N] (caller order) from the GPU + n_cpus host PEs.
+
+        Returns (scores, info): the plan and the wall time each PE took."""
+        import threading
+        import time
+
+        from .api import search_cpu
+
+        q_codes = np.ascontiguousarray(q_codes, dtype=np.uint8)
+        q_offsets = np.ascontiguousarray(q_offsets, dtype=np.int64)
+        nq = len(q_offsets) - 1
+        if plan is None:
+            plan = self.plan(np.diff(q_offsets), n_cpus, gpu_rate, cpu_rate)
+        out = np.zeros((nq, self.n_seqs), dtype=np.int32)
+        info = {"plan": plan, "cpu_s": [0.0] * plan.n_cpus, "gpu_s": 0.0}
+
+        def groups(tasks):
+            by = {}
+            for q, s in tasks:
+                by.setdefault(s, []).append(q)
+            return [(s, sorted(qs)) for s, qs in sorted(by.items())]
+
+        def cpu_pe(c):
+            t0 = time.perf_counter()
+            for s, qs in groups(plan.cpu_tasks(c)):
+                qc, qo = subset(q_codes, q_offsets, qs)
+                blk = search_cpu(qc, qo, self.host[s][0], self.host[s][1], matrix, gap_open, gap_extend,
+                                 alphabet_size=self.alphabet_size, n_threads=1)
+                out[np.ix_(qs, self.shards[s])] = blk
+            info["cpu_s"][c] = time.perf_counter() - t0
+
+        threads = [threading.Thread(target=cpu_pe, args=(c,)) for c in range(plan.n_cpus)]
+        for t in threads:
+            t.start()
+        t0 = time.perf_counter()
+        for s, qs in groups(plan.gpu_tasks(0)):
+            qc, qo = subset(q_codes, q_offsets, qs)
+            blk = np.zeros((len(qs), len(self.shards[s])), dtype=np.int32)
+            self.handle.search(qc, qo, self.gpu[s], matrix, gap_open, gap_extend, out=blk)
+            out[np.ix_(qs, self.shards[s])] = blk
+        info["gpu_s"] = time.perf_counter() - t0
+        for t in threads:
+            t.join()
+        return out, info

@@ -118,3 +118,28 @@ def test_gloo_world2_matches_single_process(n_shards):
         assert p.exitcode == 0
     for r in (0, 1):
         np.testing.assert_array_equal(outs[r], ref)
+
+
+def test_place_hybrid_cpu_and_gpu_pes():
+    """Hybrid placement: every (query, shard) task on exactly one
+    PE; CPUs get work only when their rate makes it pay; makespan <= 2 lambda
+    (Proposition 1)."""
+    from paper_conf_icpp_kedad_sidhoummmmt14_b200 import dist
+    rng = np.random.default_rng(4)
+    offs = np.zeros(2001, dtype=np.int64)
+    np.cumsum(rng.integers(10, 900, size=2000), out=offs[1:])
+    shards = dist.shard_cut(offs, 8)
+    res = [float((offs[idx + 1] - offs[idx]).sum()) for idx in shards]
+    q_lens = [144, 567, 1000, 2504, 5478]
+    slow = dist.place_hybrid(q_lens, shards, 4, 1, gpu_rate=6e12, cpu_rate=1e6, shard_residues=res)
+    assert (slow.pe == 4).all()                      # CPUs far too slow: everything on the GPU
+    mix = dist.place_hybrid(q_lens, shards, 16, 1, gpu_rate=1e11, cpu_rate=1e10, shard_residues=res)
+    assert len(mix.pe) == len(q_lens) * 8 and set(mix.pe.tolist()) <= set(range(17))
+    assert (mix.pe < 16).any() and (mix.pe == 16).any()
+    loads = np.zeros(17)
+    for t, p in enumerate(mix.pe):
+        loads[p] += mix.p_cpu[t] if p < 16 else mix.p_gpu[t]
+    assert abs(loads.max() - mix.makespan) < 1e-9 * max(1.0, mix.makespan)
+    assert mix.makespan <= 2 * mix.lam * (1 + 1e-9)
+    assert sorted(mix.cpu_tasks(0) + sum((mix.cpu_tasks(c) for c in range(1, 16)), []) + mix.gpu_tasks(0)) \
+        == sorted(mix.tasks)

@@ -280,3 +280,42 @@ def test_table5_query_sets_sampled(name):
     sub = np.concatenate([c["dcodes"][c["doff"][i]:c["doff"][i + 1]] for i in idx])
     ref = oracle_scores(c["qcodes"], c["qoff"], sub, sub_off, procs=16)
     np.testing.assert_array_equal(got[:, idx], ref)
+
+
+@pytest.mark.parametrize("gs,ge", [(0, 2), (5, 2)])
+def test_nucleotide_mode(gs, ge):
+    """DNA over ACGT(N), ma/mi scoring
+    (L127-133), linear gap of Eq. (1) as Gs = 0, Ge = -g (L159-165), and the
+    affine model, on the same kernels (alphabet 5) vs the oracle; includes the
+    Fig. 1 pair (L137-143), whose local optimum is 5."""
+    sw = _pkg()
+    rng = np.random.default_rng(44 + gs)
+    S = sw.nucleotide_matrix(1, -1)
+    q = [sw.encode_nucleotide("ACTTGTCCG"), rng.integers(0, 5, size=700).astype(np.uint8),
+         rng.integers(0, 4, size=97).astype(np.uint8)]
+    qo = np.zeros(4, dtype=np.int64)
+    np.cumsum([len(x) for x in q], out=qo[1:])
+    dl = [8] + list(rng.integers(1, 1500, size=200)) + [0, 3]
+    dc, do = _seqs(dl, rng, alpha=4)
+    dc[:8] = sw.encode_nucleotide("ATTGTCAG")
+    qc = np.concatenate(q)
+    got = gpu_scores(qc, qo, dc, do, S=S, gs=gs, ge=ge, alpha=5)
+    ref = oracle_scores(qc, qo, dc, do, S=S.astype(np.int32), gs=gs, ge=ge)
+    np.testing.assert_array_equal(got, ref)
+    if gs == 0:
+        assert got[0, 0] == 5
+
+
+def test_hybrid_cpu_gpu_search():
+    """Hybrid SWDUAL: tasks split between the GPU and 3 host
+    PEs by the dual approximation; the assembled matrix equals the oracle's."""
+    sw = _pkg()
+    from paper_conf_icpp_kedad_sidhoummmmt14_b200 import dist
+    c = swgen.make_config("c1", n_db=900)
+    qc, qo = swgen.make_queries(12, [144, 375, 60, 1000])
+    with sw.Handle(0) as h:
+        hdb = dist.HybridDB(h, c["dcodes"], c["doff"], n_shards=6)
+        got, info = hdb.search(qc, qo, sw.blosum62(), 10, 2, n_cpus=3, gpu_rate=2e10, cpu_rate=1e10)
+    plan = info["plan"]
+    assert (plan.pe < 3).any() and (plan.pe == 3).any()
+    np.testing.assert_array_equal(got, oracle_scores(qc, qo, c["dcodes"], c["doff"]))

@@ -136,6 +136,15 @@ def test_encode_ascii():
     assert got.tolist() == exp
 
 
+def test_encode_nucleotide_and_matrix():
+    got = sw.encode_nucleotide("ACGTUacgtuNnRY-")
+    assert got.tolist() == [0, 1, 2, 3, 3, 0, 1, 2, 3, 3, 4, 4, 4, 4, 4]
+    M = sw.nucleotide_matrix(1, -1)
+    assert M.shape == (5, 5) and M.dtype == np.int8
+    assert all(M[a, a] == 1 for a in range(4)) and M[4, 4] == -1
+    assert (M[~np.eye(5, dtype=bool)] == -1).all()
+
+
 def test_blosum62_tables():
     """The product's (lower-triangle) and the oracle's (full) transcriptions agree,
     and the table has BLOSUM62's known structure."""

@@ -1026,7 +1026,7 @@ int32_t sw_align(sw_handle_t h, const uint8_t* q_codes, const int64_t* q_offsets
       SW_CK(h->a_ops.ensure(size_t(std::max<int64_t>(ow, 1)) * sizeof(uint32_t)));
       SW_CK(h->a_out.ensure(size_t(nb) * 6 * sizeof(int32_t)));
       int grid = std::min(nb, h->sms * 4);
-      const int64_t link_budget = int64_t(256) << 20;  // bytes of warp link rows
+      const int64_t link_budget = int64_t(1) << 30;  // bytes of warp link rows (HBM is plentiful)
       const int64_t per_cta = int64_t(ALIGN_WARPS) * bcap * int64_t(sizeof(int2));
       grid = int(std::max<int64_t>(1, std::min<int64_t>(grid, std::max<int64_t>(h->sms, link_budget / per_cta))));
       SW_CK(h->a_links.ensure(size_t(grid) * size_t(per_cta)));

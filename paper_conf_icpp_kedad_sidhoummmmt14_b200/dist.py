@@ -181,12 +181,20 @@ class HybridPlan:
 def place_hybrid(q_lens, shards, n_cpus: int, n_gpus: int, gpu_rate: float, cpu_rate: float,
                  shard_residues=None) -> HybridPlan:
     """Tasks (query, shard) with p = cells / rate on each PE type (reading S-1/S-2),
-    placed by the dual approximation on n_cpus CPU PEs + n_gpus GPUs."""
+    placed by the dual approximation on n_cpus CPU PEs + n_gpus GPUs.
+
+    gpu_rate / cpu_rate: cells per second, a scalar or one value per query (the
+    GPU's rate depends on the query length -- short queries fill its lanes
+    worse -- so p_cpu / p_gpu differs between tasks, which is what the
+    knapsack of the dual approximation orders by, L370-387)."""
     if shard_residues is None:
         raise ValueError("shard_residues required")
     tasks = [(q, s) for q in range(len(q_lens)) for s in range(len(shards))]
     cells = np.array([float(q_lens[q]) * float(shard_residues[s]) for q, s in tasks], dtype=np.float64)
-    p_cpu, p_gpu = cells / float(cpu_rate), cells / float(gpu_rate)
+    qi = np.array([q for q, _ in tasks], dtype=np.int64)
+    gr = np.broadcast_to(np.asarray(gpu_rate, dtype=np.float64), (len(q_lens),))[qi] if tasks else np.zeros(0)
+    cr = np.broadcast_to(np.asarray(cpu_rate, dtype=np.float64), (len(q_lens),))[qi] if tasks else np.zeros(0)
+    p_cpu, p_gpu = cells / cr, cells / gr
     if tasks:
         pe, mk, lam = schedule_dual(p_cpu, p_gpu, n_cpus, n_gpus)
     else:

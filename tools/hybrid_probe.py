@@ -29,18 +29,32 @@ plan0 = hdb.plan(qlen, 0, 1.0, 1.0)
 hdb.search(c["qcodes"], c["qoff"], S, plan=plan0)
 t = time.perf_counter(); ref, _ = hdb.search(c["qcodes"], c["qoff"], S, plan=plan0); t_gpu = time.perf_counter() - t
 gpu_rate = cells / t_gpu
+# per-query GPU rates (the GPU's cell rate depends on the query length)
+db_full = h.load_db(c["dcodes"], c["doff"])
+rates = []
+for q in range(len(qlen)):
+    qq, oo = c["qcodes"][c["qoff"][q]:c["qoff"][q + 1]], np.array([0, qlen[q]], dtype=np.int64)
+    out = torch.empty((1, db_full.n_seqs), dtype=torch.int32, device="cuda")
+    h.search(qq, oo, db_full, S, 10, 2, out=out)
+    torch.cuda.synchronize()
+    t = time.perf_counter()
+    h.search(qq, oo, db_full, S, 10, 2, out=out)
+    torch.cuda.synchronize()
+    rates.append(float(qlen[q]) * float(c["doff"][-1] - c["doff"][0]) / (time.perf_counter() - t))
+db_full.free()
+gpu_rate_q = np.array(rates) * (gpu_rate / (cells / sum(float(qlen[q]) * float(c["doff"][-1] - c["doff"][0]) / rates[q] for q in range(len(qlen)))))
 sl = hdb.host[0]
 k = min(len(sl[1]) - 1, 3000)
 qc, qo = swgen.make_queries(5, [567])
 t = time.perf_counter()
 sw.search_cpu(qc, qo, sl[0][:sl[1][k] - sl[1][0]], sl[1][:k + 1] - sl[1][0], S, 10, 2, n_threads=1)
 cpu_rate = 567.0 * float(sl[1][k] - sl[1][0]) / (time.perf_counter() - t)
-plan = hdb.plan(qlen, n_cpus, gpu_rate, cpu_rate)
+plan = hdb.plan(qlen, n_cpus, gpu_rate_q, cpu_rate)
 hdb.search(c["qcodes"], c["qoff"], S, plan=plan)
 t = time.perf_counter(); got, info = hdb.search(c["qcodes"], c["qoff"], S, plan=plan); t_hyb = time.perf_counter() - t
 cpu_cells = sum(float(qlen[q]) * hdb.residues[s] for (q, s), p in zip(plan.tasks, plan.pe) if p < n_cpus)
 print(json.dumps({"workload": wl, "shards": n_shards, "tasks": len(plan.tasks), "host_cores": cores, "cpu_pes": n_cpus,
-                  "gpu_rate_GCUPS": round(gpu_rate / 1e9, 1), "cpu_pe_rate_GCUPS": round(cpu_rate / 1e9, 2),
+                  "gpu_rate_GCUPS": round(gpu_rate / 1e9, 1), "gpu_rate_per_query_GCUPS": [round(r / 1e9) for r in gpu_rate_q], "cpu_pe_rate_GCUPS": round(cpu_rate / 1e9, 2),
                   "gpu_only_s": round(t_gpu, 4), "hybrid_s": round(t_hyb, 4),
                   "hybrid_GCUPS": round(cells / t_hyb / 1e9, 1), "gpu_only_GCUPS": round(cells / t_gpu / 1e9, 1),
                   "tasks_on_cpus": int((plan.pe < n_cpus).sum()), "cell_share_on_cpus": round(cpu_cells / cells, 5),

@@ -133,6 +133,13 @@ __device__ __forceinline__ void copy_strip(uint8_t* dst, const uint8_t* __restri
 #ifndef SW_CODES
 #define SW_CODES 0
 #endif
+// SW_Q2_ADDR 1: lane 0 turns the DB letter into its profile-row address once per
+// column (PRMT + IMAD) and the lanes shuffle addresses instead of codes: 2 fewer
+// ALU ops per column, but the extra live register doubles the spill at the
+// 128-register cap -- measured -7.5% on config 3 (+0.4% on config 2); kept off.
+#ifndef SW_Q2_ADDR
+#define SW_Q2_ADDR 0
+#endif
 #ifndef SW_BB_HINT
 #define SW_BB_HINT 0
 #endif
@@ -179,15 +186,20 @@ __device__ __forceinline__ void strip_pass(const uint8_t* sprof, int LS, int LB,
   uint32_t HA[R], E[R];
 #pragma unroll
   for (int r = 0; r < R; ++r) { HA[r] = 0; E[r] = 0; }
-  uint32_t hdiag = 0, sH = 0, sF = 0, sC = code_pad2;
+  const uint32_t sbase = static_cast<uint32_t>(__cvta_generic_to_shared(sprof));
+  // Q2 (SW_Q2_ADDR): the code that travels down the lanes is already the shared
+  // address of the DB letter's profile row (lane-independent); lane 0 forms it
+  // once per column with one PRMT (byte select) + IMAD, the others add laneoff.
+  const uint32_t c0pad = (Q2 && SW_Q2_ADDR) ? sbase + (code_pad2 & 0xffu) * LS : code_pad2;
+  uint32_t hdiag = 0, sH = 0, sF = 0, sC = c0pad;
   const uint2* __restrict__ codes = reinterpret_cast<const uint2*>(pstream);
   const uint32_t pad4 = code_pad2 | (code_pad2 << 16);
   const uint32_t laneoff = uint32_t(k) * LB;
   const bool lead = (k == 0), tail = (k == G - 1);
   const uint2 z2 = make_uint2(0, 0);
   // second sub-lane: its inputs are the first sub-lane's outputs of the previous step
-  uint32_t hdiag1 = 0, cH = 0, cF = 0, pC = code_pad2;
-  const uint32_t sbase = static_cast<uint32_t>(__cvta_generic_to_shared(sprof));
+  uint32_t hdiag1 = 0, cH = 0, cF = 0, pC = c0pad;
+  const uint32_t bsel = (shift >> 3) | 0x4440u;  // PRMT selector: byte `shift/8` of a column word, zero-extended
   const uint32_t pad_row = sbase + (code_pad2 & 0xffu) * LS + laneoff;
   uint32_t ppa = pad_row, ppb = pad_row;
   rp += VG - 1;  // sub-lane 0 of lane 0 reads column c at rp[c + VG - 1]
@@ -240,13 +252,17 @@ __device__ __forceinline__ void strip_pass(const uint8_t* sprof, int LS, int LB,
       uint32_t rC = __shfl_up_sync(FULL, sC, 1, G);
       if (lead) {
         const uint32_t w = (j < 2) ? cwc.x : cwc.y;
-        rC = (j & 1) ? (w >> 16) : (w & 0xffffu);
+        if constexpr (Q2 && SW_Q2_ADDR) rC = sbase + prmt(w, 0u, bsel + ((j & 1) ? 2u : 0u)) * LS;
+        else rC = (j & 1) ? (w >> 16) : (w & 0xffffu);
         const uint2 tv = (j == 0) ? c0 : (j == 1) ? c1 : (j == 2) ? c2 : c3;
         rH = tv.x;
         rF = tv.y;
       }
       uint32_t pa, pb;
-      if constexpr (Q2) {  // one DB sequence (byte `shift` of the pair word) against two queries
+      if constexpr (Q2 && SW_Q2_ADDR) {  // rC = profile-row address of the DB letter
+        pa = rC + laneoff;
+        pb = pa;
+      } else if constexpr (Q2) {  // one DB sequence (byte `shift` of the pair word) against two queries
         pa = sbase + ((rC >> shift) & 0xffu) * LS + laneoff;
         pb = pa;
       } else {
@@ -317,7 +333,11 @@ __device__ __forceinline__ void emit_pair(const InterArgs& a, const QueryDesc& d
 //     (inter-task mode).
 // Queries are in descending length, pairs in descending length.
 template <int G, int R, int NT>
+#ifdef SW_MINB  // experiments only: __launch_bounds__(NT, 1) lets ptxas take 225 registers (1 CTA/SM, -5% on config 3)
+__global__ void __launch_bounds__(NT, SW_MINB) inter_kernel(InterArgs a) {
+#else
 __global__ void __launch_bounds__(NT) inter_kernel(InterArgs a) {
+#endif
   extern __shared__ __align__(16) uint8_t smem[];
   // An item is either short or long, so the two uses share shared memory:
   uint8_t* sprof = smem;                         // short mode: the strip profile (bank-spread copies)

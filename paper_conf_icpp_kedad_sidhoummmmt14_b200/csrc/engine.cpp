@@ -1057,11 +1057,6 @@ int32_t sw_align(sw_handle_t h, const uint8_t* q_codes, const int64_t* q_offsets
       SW_CK(cudaMemcpyAsync(hout.data(), h->a_out.p, hout.size() * sizeof(int32_t), cudaMemcpyDeviceToHost, st));
       if (ow) SW_CK(cudaMemcpyAsync(hops.data(), h->a_ops.p, size_t(ow) * sizeof(uint32_t), cudaMemcpyDeviceToHost, st));
       SW_CK(cudaStreamSynchronize(st));
-      if (const char* dump = std::getenv("SWDUAL_ALIGN_DUMP")) {  // debugging aid: raw traceback codes
-        std::vector<uint32_t> tr(static_cast<size_t>(tw));
-        SW_CK(cudaMemcpy(tr.data(), h->a_trace.p, size_t(tw) * 4, cudaMemcpyDeviceToHost));
-        if (FILE* f = std::fopen(dump, "wb")) { std::fwrite(tr.data(), 4, tr.size(), f); std::fclose(f); }
-      }
       for (int x = 0; x < nb; ++x) {
         const AlignItem& it = items[b0 + size_t(x)];
         const int32_t k = item_pair[b0 + size_t(x)];

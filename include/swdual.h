@@ -226,6 +226,21 @@ int32_t sw_schedule_dual(int64_t n_tasks, const double* p_cpu, const double* p_g
                          int32_t n_gpu, int32_t* out_pe, double* out_makespan, double* out_lambda);
 
 /*
+ * The dynamic-programming variant of the same binary search (PAPER.md L482-502:
+ * counting the tasks "with processing times larger than" a fraction of lambda and
+ * solving the knapsack "via dynamic programming" brings the guarantee towards
+ * 3/2 OPT; reading S-8).  Per guess: a task is big on a side when it
+ * takes > lambda/2 there; the DP assigns sides minimising the CPU area with at
+ * most n_cpu CPU-big and n_gpu GPU-big tasks and GPU area <= n_gpu * lambda (GPU
+ * times rounded down to lambda / (4 n_tasks)); LPT on each side.  Makespan
+ * <= (3/2 + 1/(4 n_gpu)) * lambda.  Same arguments and outputs as
+ * sw_schedule_dual.  Time O(n^2 m k^2) per guess: SW_EUNSUPPORTED when the DP
+ * would exceed ~4e9 state updates.
+ */
+int32_t sw_schedule_dual_dp(int64_t n_tasks, const double* p_cpu, const double* p_gpu, int32_t n_cpu,
+                            int32_t n_gpu, int32_t* out_pe, double* out_makespan, double* out_lambda);
+
+/*
  * Host packer only (no device work): the packed form sw_load_db uploads.
  * Non-empty sequences sorted by length (longest first, ties by index), paired
  * neighbours (id1 = -1 for an odd leftover), each pair interleaved into 16-bit

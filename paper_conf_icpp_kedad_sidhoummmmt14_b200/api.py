@@ -207,13 +207,16 @@ def encode_nucleotide(s: str) -> np.ndarray:
     return out
 
 
-def schedule_dual(p_cpu, p_gpu, n_cpu: int, n_gpu: int):
-    """sw_schedule_dual: (pe int32[n], makespan, lambda); PEs 0..n_cpu-1 are CPUs, then GPUs."""
+def schedule_dual(p_cpu, p_gpu, n_cpu: int, n_gpu: int, variant: str = "greedy"):
+    """sw_schedule_dual (variant "greedy": the 2-approximation) or sw_schedule_dual_dp
+    (variant "dp": the DP-knapsack refinement): (pe int32[n], makespan, lambda);
+    PEs 0..n_cpu-1 are CPUs, then GPUs."""
     pc = _host(p_cpu, np.float64)
     pg = _host(p_gpu, np.float64)
     n = len(pc)
     pe = np.full(n, -1, dtype=np.int32)
     mk, lam = ctypes.c_double(), ctypes.c_double()
-    check(lib().sw_schedule_dual(n, _vp(pc) if n else None, _vp(pg) if n else None, int(n_cpu), int(n_gpu),
+    fn = {"greedy": lib().sw_schedule_dual, "dp": lib().sw_schedule_dual_dp}[variant]
+    check(fn(n, _vp(pc) if n else None, _vp(pg) if n else None, int(n_cpu), int(n_gpu),
                                  _vp(pe) if n else None, ctypes.byref(mk), ctypes.byref(lam)))
     return pe, mk.value, lam.value

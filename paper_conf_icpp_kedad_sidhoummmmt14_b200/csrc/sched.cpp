@@ -18,6 +18,7 @@
 // method reduces to binary search + LPT list scheduling.
 #include <algorithm>
 #include <cmath>
+#include <limits>
 #include <cstdint>
 #include <numeric>
 #include <vector>
@@ -78,10 +79,85 @@ bool dual_step(int64_t n, const double* pc, const double* pg, int m, int k, doub
   return true;
 }
 
+// One step of the DP-knapsack variant for guess lam ("constraints
+// on the number of tasks with processing times larger than" a fraction of lambda,
+// solved "via dynamic programming", after [13]; reading S-8).  A task is
+// big on a side when it takes more than lam/2 there; a schedule of makespan <= lam
+// holds at most m big tasks on the CPUs and k on the GPUs.  The DP chooses the side
+// of every task minimising the CPU area under those counts and the GPU area <= k*lam
+// (GPU times rounded down to lam/(4n): a feasible lam is never rejected).  Then LPT
+// list scheduling on each side: the bigs land alone first, any later task starts
+// below the average load, so CPUs end by 3/2 lam and GPUs by (3/2 + 1/(4k)) lam.
+bool dual_step_dp(int64_t n, const double* pc, const double* pg, int m, int k, double lam, Sched& out) {
+  constexpr int GRID = 4;
+  out.pe.assign(size_t(n), -1);
+  const double half = 0.5 * lam;
+  const double delta = lam / (double(GRID) * double(n));
+  const int64_t cap = k > 0 ? int64_t(k) * GRID * n : 0;
+  const int64_t M1 = m + 1, K1 = k + 1, C1 = cap + 1;
+  const int64_t S = M1 * K1 * C1;
+  const double INF = std::numeric_limits<double>::infinity();
+  std::vector<double> cur(static_cast<size_t>(S), INF), nxt(static_cast<size_t>(S), INF);
+  std::vector<uint8_t> choice(size_t(n) * size_t(S), 0);  // 1 = task on a GPU
+  cur[0] = 0.0;
+  auto idx = [&](int64_t mu, int64_t ka, int64_t g) { return (mu * K1 + ka) * C1 + g; };
+  for (int64_t j = 0; j < n; ++j) {
+    std::fill(nxt.begin(), nxt.end(), INF);
+    const bool cpu_ok = m > 0 && pc[j] <= lam, gpu_ok = k > 0 && pg[j] <= lam;
+    if (!cpu_ok && !gpu_ok) return false;
+    const int bc = pc[j] > half ? 1 : 0, bg = pg[j] > half ? 1 : 0;
+    const int64_t r = gpu_ok ? int64_t(std::floor(pg[j] / delta)) : 0;
+    uint8_t* ch = choice.data() + size_t(j) * size_t(S);
+    for (int64_t mu = 0; mu < M1; ++mu)
+      for (int64_t ka = 0; ka < K1; ++ka)
+        for (int64_t g = 0; g < C1; ++g) {
+          const double w = cur[size_t(idx(mu, ka, g))];
+          if (w == INF) continue;
+          if (cpu_ok && mu + bc < M1) {
+            const int64_t t = idx(mu + bc, ka, g);
+            if (w + pc[j] < nxt[size_t(t)]) { nxt[size_t(t)] = w + pc[j]; ch[t] = 0; }
+          }
+          if (gpu_ok && ka + bg < K1 && g + r < C1) {
+            const int64_t t = idx(mu, ka + bg, g + r);
+            if (w < nxt[size_t(t)]) { nxt[size_t(t)] = w; ch[t] = 1; }
+          }
+        }
+    cur.swap(nxt);
+  }
+  int64_t bst = -1;
+  for (int64_t t = 0; t < S; ++t)
+    if (cur[size_t(t)] != INF && (bst < 0 || cur[size_t(t)] < cur[size_t(bst)])) bst = t;
+  if (bst < 0 || cur[size_t(bst)] > m * lam + 1e-12 * std::max(1.0, cur[size_t(bst)])) return false;
+  // walk the choices back from the best final state
+  std::vector<int64_t> cpu, gpu;
+  int64_t mu = bst / (K1 * C1), ka = (bst / C1) % K1, g = bst % C1;
+  for (int64_t j = n - 1; j >= 0; --j) {
+    const int64_t t = idx(mu, ka, g);
+    if (choice[size_t(j) * size_t(S) + size_t(t)]) {
+      gpu.push_back(j);
+      ka -= pg[j] > half ? 1 : 0;
+      g -= int64_t(std::floor(pg[j] / delta));
+    } else {
+      cpu.push_back(j);
+      mu -= pc[j] > half ? 1 : 0;
+    }
+  }
+  const double mc = list_schedule(cpu, pc, m, 0, out.pe);
+  const double mg = list_schedule(gpu, pg, k, m, out.pe);
+  out.makespan = std::max(mc, mg);
+  return true;
+}
+
+using step_fn = bool (*)(int64_t, const double*, const double*, int, int, double, Sched&);
+
+int32_t binary_search(step_fn step, int64_t n_tasks, const double* p_cpu, const double* p_gpu, int32_t n_cpu,
+                      int32_t n_gpu, int32_t* out_pe, double* out_makespan, double* out_lambda);
+
 }  // namespace
 
-extern "C" int32_t sw_schedule_dual(int64_t n_tasks, const double* p_cpu, const double* p_gpu, int32_t n_cpu,
-                                    int32_t n_gpu, int32_t* out_pe, double* out_makespan, double* out_lambda) {
+namespace {
+int32_t binary_search(step_fn step, int64_t n_tasks, const double* p_cpu, const double* p_gpu, int32_t n_cpu,
+                      int32_t n_gpu, int32_t* out_pe, double* out_makespan, double* out_lambda) {
   if (n_tasks < 0 || n_cpu < 0 || n_gpu < 0 || n_cpu + n_gpu < 1) return SW_EINVAL;
   if (n_tasks > 0 && (!p_cpu || !p_gpu || !out_pe)) return SW_EINVAL;
   for (int64_t j = 0; j < n_tasks; ++j)
@@ -108,12 +184,12 @@ extern "C" int32_t sw_schedule_dual(int64_t n_tasks, const double* p_cpu, const 
   // the list schedule on the faster side per task, then double until accepted.
   Sched best, cur;
   double hi = std::max(lo, 1e-300);
-  while (!dual_step(n_tasks, p_cpu, p_gpu, m, k, hi, cur)) hi *= 2;
+  while (!step(n_tasks, p_cpu, p_gpu, m, k, hi, cur)) hi *= 2;
   best = cur;
   double lam_acc = hi;
   for (int it = 0; it < 64 && hi - lo > 1e-4 * hi; ++it) {
     const double lam = 0.5 * (lo + hi);
-    if (dual_step(n_tasks, p_cpu, p_gpu, m, k, lam, cur)) {
+    if (step(n_tasks, p_cpu, p_gpu, m, k, lam, cur)) {
       hi = lam;
       lam_acc = lam;
       if (cur.makespan <= best.makespan) best = cur;
@@ -125,4 +201,18 @@ extern "C" int32_t sw_schedule_dual(int64_t n_tasks, const double* p_cpu, const 
   if (out_makespan) *out_makespan = best.makespan;
   if (out_lambda) *out_lambda = lam_acc;
   return SW_OK;
+}
+}  // namespace
+
+extern "C" int32_t sw_schedule_dual(int64_t n_tasks, const double* p_cpu, const double* p_gpu, int32_t n_cpu,
+                                    int32_t n_gpu, int32_t* out_pe, double* out_makespan, double* out_lambda) {
+  return binary_search(dual_step, n_tasks, p_cpu, p_gpu, n_cpu, n_gpu, out_pe, out_makespan, out_lambda);
+}
+
+extern "C" int32_t sw_schedule_dual_dp(int64_t n_tasks, const double* p_cpu, const double* p_gpu, int32_t n_cpu,
+                                       int32_t n_gpu, int32_t* out_pe, double* out_makespan, double* out_lambda) {
+  // the DP table holds (m+1)(k+1)(4kn+1) states per task
+  const double states = double(n_cpu + 1) * double(n_gpu + 1) * (4.0 * double(n_gpu) * double(n_tasks) + 1.0);
+  if (n_tasks > 0 && states * double(n_tasks) > 4.0e9) return SW_EUNSUPPORTED;
+  return binary_search(dual_step_dp, n_tasks, p_cpu, p_gpu, n_cpu, n_gpu, out_pe, out_makespan, out_lambda);
 }

@@ -84,3 +84,49 @@ def test_task_longer_than_lambda_goes_to_other_side():
     # task 0 is hopeless on the CPU, task 1 on the GPU: a 1+1 box must split them
     pe, mk, lam = schedule_dual([100.0, 1.0], [1.0, 100.0], 1, 1)
     assert pe.tolist() == [1, 0] and mk == pytest.approx(1.0)
+
+
+@pytest.mark.parametrize("seed", range(6))
+def test_dp_variant_vs_brute_force(seed):
+    """DP-knapsack variant (reading S-8): every lambda >= OPT is
+    accepted and the schedule ends by (3/2 + 1/(4k)) lambda, so it is within that
+    factor of the brute-force optimum."""
+    rng = np.random.default_rng(100 + seed)
+    for _ in range(25):
+        n = int(rng.integers(1, 7))
+        m = int(rng.integers(0, 3))
+        k = int(rng.integers(1, 3))
+        if m + k > 3:
+            continue
+        pg = rng.uniform(0.1, 10.0, n)
+        pc = pg * rng.uniform(0.5, 30.0, n)
+        pe, mk, lam = schedule_dual(pc, pg, m, k, variant="dp")
+        assert np.all((pe >= 0) & (pe < m + k))
+        L = loads(pe, pc, pg, m, k)
+        assert mk == pytest.approx(L.max())
+        bound = 1.5 + 0.25 / k
+        assert mk <= bound * lam * (1 + 1e-9)
+        opt = brute_opt(pc, pg, m, k)
+        assert lam <= opt * (1 + 2e-4) + 1e-12
+        assert mk <= bound * opt * (1 + 2e-4) + 1e-12
+
+
+def test_dp_variant_not_worse_on_average():
+    """On random hybrid instances the DP variant's makespans are on average no
+    worse than the greedy 2-approximation's (same binary search)."""
+    rng = np.random.default_rng(77)
+    ratios = []
+    for _ in range(40):
+        n, m, k = int(rng.integers(8, 30)), int(rng.integers(1, 6)), int(rng.integers(1, 3))
+        pg = rng.uniform(1, 20, n)
+        pc = pg * rng.uniform(2, 20, n)
+        _, mg, _ = schedule_dual(pc, pg, m, k)
+        _, md, _ = schedule_dual(pc, pg, m, k, variant="dp")
+        ratios.append(md / mg)
+    assert np.mean(ratios) <= 1.0 + 1e-9
+
+
+def test_dp_variant_size_limit():
+    pg = np.ones(5000)
+    with pytest.raises(SWError):
+        schedule_dual(pg * 3, pg, 64, 8, variant="dp")

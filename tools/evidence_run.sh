@@ -1,6 +1,6 @@
 #!/bin/bash
 # One GPU call that refreshes the round's committed evidence (run under gpurun).
-# Outputs land in gpurun_out/ev_*; tools/evidence_collect.py turns them into profiles/.
+# Outputs land in gpurun_out/ev_*; tools/ncu_summary.py turns the ncu files into profiles/ summaries.
 set -x
 mkdir -p gpurun_out
 nvidia-smi --query-gpu=name,clocks.sm,clocks.max.sm,power.draw --format=csv > gpurun_out/ev_smi.txt

@@ -137,6 +137,18 @@ __device__ __forceinline__ void copy_strip(uint8_t* dst, const uint8_t* __restri
 // column (PRMT + IMAD) and the lanes shuffle addresses instead of codes: 2 fewer
 // ALU ops per column, but the extra live register doubles the spill at the
 // 128-register cap -- measured -7.5% on config 3 (+0.4% on config 2); kept off.
+// SW_SEL_IMAD 1: lane 0's three per-column selects (code, H, F of the row above)
+// as integer multiply-adds (FMA pipe) instead of SEL (ALU pipe).
+#ifndef SW_SEL_IMAD
+#define SW_SEL_IMAD 0
+#endif
+// a == 1 ? v : x, as x + a * (v - x) in two IMADs (a in {0, 1}; exact mod 2^32)
+__device__ __forceinline__ uint32_t fma_sel(uint32_t a, uint32_t v, uint32_t x) {
+  uint32_t d, r;
+  asm("mad.lo.u32 %0, %1, 1, %2;" : "=r"(d) : "r"(v), "r"(0u - x));
+  asm("mad.lo.u32 %0, %1, %2, %3;" : "=r"(r) : "r"(a), "r"(d), "r"(x));
+  return r;
+}
 #ifndef SW_Q2_ADDR
 #define SW_Q2_ADDR 0
 #endif
@@ -196,6 +208,9 @@ __device__ __forceinline__ void strip_pass(const uint8_t* sprof, int LS, int LB,
   const uint32_t pad4 = code_pad2 | (code_pad2 << 16);
   const uint32_t laneoff = uint32_t(k) * LB;
   const bool lead = (k == 0), tail = (k == G - 1);
+#if SW_SEL_IMAD
+  const uint32_t lead01 = lead ? 1u : 0u;
+#endif
   const uint2 z2 = make_uint2(0, 0);
   // second sub-lane: its inputs are the first sub-lane's outputs of the previous step
   uint32_t hdiag1 = 0, cH = 0, cF = 0, pC = c0pad;
@@ -250,6 +265,16 @@ __device__ __forceinline__ void strip_pass(const uint8_t* sprof, int LS, int LB,
       uint32_t rH = __shfl_up_sync(FULL, sH, 1, G);
       uint32_t rF = __shfl_up_sync(FULL, sF, 1, G);
       uint32_t rC = __shfl_up_sync(FULL, sC, 1, G);
+#if SW_SEL_IMAD
+      {  // lane 0 takes the boundary row: x + lead01 * (v - x) on the FMA pipe instead of SEL (ALU)
+        const uint32_t w = (j < 2) ? cwc.x : cwc.y;
+        const uint32_t cl = (j & 1) ? (w >> 16) : (w & 0xffffu);
+        const uint2 tv = (j == 0) ? c0 : (j == 1) ? c1 : (j == 2) ? c2 : c3;
+        rC = fma_sel(lead01, cl, rC);
+        rH = fma_sel(lead01, tv.x, rH);
+        rF = fma_sel(lead01, tv.y, rF);
+      }
+#else
       if (lead) {
         const uint32_t w = (j < 2) ? cwc.x : cwc.y;
         if constexpr (Q2 && SW_Q2_ADDR) rC = sbase + prmt(w, 0u, bsel + ((j & 1) ? 2u : 0u)) * LS;
@@ -258,6 +283,7 @@ __device__ __forceinline__ void strip_pass(const uint8_t* sprof, int LS, int LB,
         rH = tv.x;
         rF = tv.y;
       }
+#endif
       uint32_t pa, pb;
       if constexpr (Q2 && SW_Q2_ADDR) {  // rC = profile-row address of the DB letter
         pa = rC + laneoff;

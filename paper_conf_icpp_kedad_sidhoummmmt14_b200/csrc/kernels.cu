@@ -138,7 +138,13 @@ __device__ __forceinline__ void copy_strip(uint8_t* dst, const uint8_t* __restri
 // ALU ops per column, but the extra live register doubles the spill at the
 // 128-register cap -- measured -7.5% on config 3 (+0.4% on config 2); kept off.
 // SW_SEL_IMAD 1: lane 0's three per-column selects (code, H, F of the row above)
-// as integer multiply-adds (FMA pipe) instead of SEL (ALU pipe).
+// as integer multiply-adds (FMA pipe) instead of SEL (ALU pipe).  Measured -2% on
+// config 3 (+0.8% on config 4): one ALU op traded for two issue slots; kept off.
+// SW_T0_UNROLL: unroll factor of the 4-column block loop of a strip pass (2 measured
+// -1.4% on config 3: more register moves and spill; kept at 1)
+#ifndef SW_T0_UNROLL
+#define SW_T0_UNROLL 1
+#endif
 #ifndef SW_SEL_IMAD
 #define SW_SEL_IMAD 0
 #endif
@@ -239,6 +245,9 @@ __device__ __forceinline__ void strip_pass(const uint8_t* sprof, int LS, int LB,
     }
   }
   __syncwarp();
+#if SW_T0_UNROLL == 2
+#pragma unroll 2
+#endif
   for (int t0 = 0; t0 < T; t0 += 4) {
     const uint2 cwc = cw;
     const uint2 c0 = tb0, c1 = tb1, c2 = tb2, c3 = tb3;

@@ -179,7 +179,7 @@ class HybridPlan:
 
 
 def place_hybrid(q_lens, shards, n_cpus: int, n_gpus: int, gpu_rate: float, cpu_rate: float,
-                 shard_residues=None) -> HybridPlan:
+                 shard_residues=None, variant: str = "greedy") -> HybridPlan:
     """Tasks (query, shard) with p = cells / rate on each PE type (reading S-1/S-2),
     placed by the dual approximation on n_cpus CPU PEs + n_gpus GPUs.
 
@@ -196,7 +196,7 @@ def place_hybrid(q_lens, shards, n_cpus: int, n_gpus: int, gpu_rate: float, cpu_
     cr = np.broadcast_to(np.asarray(cpu_rate, dtype=np.float64), (len(q_lens),))[qi] if tasks else np.zeros(0)
     p_cpu, p_gpu = cells / cr, cells / gr
     if tasks:
-        pe, mk, lam = schedule_dual(p_cpu, p_gpu, n_cpus, n_gpus)
+        pe, mk, lam = schedule_dual(p_cpu, p_gpu, n_cpus, n_gpus, variant=variant)
     else:
         pe, mk, lam = np.zeros(0, np.int32), 0.0, 0.0
     return HybridPlan(shards, tasks, np.asarray(pe, np.int64), n_cpus, n_gpus, mk, lam, p_cpu, p_gpu)
@@ -216,8 +216,9 @@ class HybridDB:
         self.gpu = [handle.load_db(c, o, alphabet_size=alphabet_size) for c, o in self.host]
         self.residues = [float(o[-1] - o[0]) for _, o in self.host]
 
-    def plan(self, q_lens, n_cpus: int, gpu_rate: float, cpu_rate: float) -> HybridPlan:
-        return place_hybrid(q_lens, self.shards, n_cpus, 1, gpu_rate, cpu_rate, shard_residues=self.residues)
+    def plan(self, q_lens, n_cpus: int, gpu_rate: float, cpu_rate: float, variant: str = "greedy") -> HybridPlan:
+        return place_hybrid(q_lens, self.shards, n_cpus, 1, gpu_rate, cpu_rate, shard_residues=self.residues,
+                            variant=variant)
 
     def search(self, q_codes, q_offsets, matrix, gap_open=10, gap_extend=2, n_cpus: int = 4,
                gpu_rate: float = 6.5e12, cpu_rate: float = 3.0e9, plan: HybridPlan | None = None):

@@ -143,3 +143,18 @@ def test_place_hybrid_cpu_and_gpu_pes():
     assert mix.makespan <= 2 * mix.lam * (1 + 1e-9)
     assert sorted(mix.cpu_tasks(0) + sum((mix.cpu_tasks(c) for c in range(1, 16)), []) + mix.gpu_tasks(0)) \
         == sorted(mix.tasks)
+
+
+def test_place_hybrid_dp_variant():
+    from paper_conf_icpp_kedad_sidhoummmmt14_b200 import dist
+    rng = np.random.default_rng(5)
+    offs = np.zeros(301, dtype=np.int64)
+    np.cumsum(rng.integers(10, 900, size=300), out=offs[1:])
+    shards = dist.shard_cut(offs, 4)
+    res = [float((offs[idx + 1] - offs[idx]).sum()) for idx in shards]
+    q_lens = [144, 567, 1000]
+    g = dist.place_hybrid(q_lens, shards, 3, 1, gpu_rate=5e9, cpu_rate=1e9, shard_residues=res)
+    d = dist.place_hybrid(q_lens, shards, 3, 1, gpu_rate=5e9, cpu_rate=1e9, shard_residues=res, variant="dp")
+    assert len(d.pe) == len(g.pe) == 12
+    assert d.makespan <= (1.5 + 0.25) * d.lam * (1 + 1e-9)
+    assert d.makespan <= 2 * g.makespan

@@ -143,3 +143,24 @@ def test_align_edges_and_errors():
                         vp(offs), vp(nops), None)
         ref = oracle.gotoh_align(q, d, S2.astype(np.int32), 0, 1)
         assert len(ref[5]) > 1 and rc == sw._lib.SW_EINVAL
+
+
+def test_align_nucleotides_fig1_and_random():
+    """Nucleotide mode (alphabet 5, ma/mi, Gs = 0 linear gap of Eq. (1)): the
+    Fig. 1 pair and random DNA with many ties."""
+    sw = _pkg()
+    rng = np.random.default_rng(21)
+    S = sw.nucleotide_matrix(1, -1)
+    qs = [sw.encode_nucleotide("ACTTGTCCG"), rng.integers(0, 4, size=300).astype(np.uint8),
+          rng.integers(0, 5, size=1100).astype(np.uint8)]
+    qo = np.zeros(len(qs) + 1, dtype=np.int64)
+    np.cumsum([len(x) for x in qs], out=qo[1:])
+    qc = np.concatenate(qs)
+    dl = [8, 250, 901, 33, 1]
+    dc, do = _seqs(dl, rng, 4)
+    dc[:8] = sw.encode_nucleotide("ATTGTCAG")
+    pairs = [(q, d) for q in range(len(qs)) for d in range(len(dl))]
+    for gs, ge in ((0, 2), (3, 1)):
+        _check(qc, qo, dc, do, pairs, S.astype(np.int32), gs, ge, 5)
+    got = _run(qc, qo, dc, do, [(0, 0)], S, 0, 2, 5)
+    assert got[0][0] == 5

@@ -316,6 +316,9 @@ def test_hybrid_cpu_gpu_search():
     with sw.Handle(0) as h:
         hdb = dist.HybridDB(h, c["dcodes"], c["doff"], n_shards=6)
         got, info = hdb.search(qc, qo, sw.blosum62(), 10, 2, n_cpus=3, gpu_rate=2e10, cpu_rate=1e10)
+        plan_dp = hdb.plan(np.diff(qo), 3, 2e10, 1e10, variant="dp")
+        got_dp, _ = hdb.search(qc, qo, sw.blosum62(), 10, 2, plan=plan_dp)
     plan = info["plan"]
     assert (plan.pe < 3).any() and (plan.pe == 3).any()
     np.testing.assert_array_equal(got, oracle_scores(qc, qo, c["dcodes"], c["doff"]))
+    np.testing.assert_array_equal(got_dp, got)

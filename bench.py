@@ -63,7 +63,7 @@ def parse():
     ap.add_argument("--impl", default="ours", choices=["ours", "reference"])
     ap.add_argument("--workload", default="c3", choices=sorted(WORKLOADS))
     ap.add_argument("--n-db", type=int, default=None, help="override DB size (smoke runs only)")
-    ap.add_argument("--e2e-steps", type=int, default=2)
+    ap.add_argument("--e2e-steps", type=int, default=3)
     ap.add_argument("--no-cpu-baseline", action="store_true")
     ap.add_argument("--cpu-baseline-cells", type=float, default=3.0e10)
     ap.add_argument("--force-geom", default=None, help="G,R of the inter-task kernel (experiments; default auto)")
@@ -359,10 +359,7 @@ def run_ours(args):
         final_host = torch.empty(world * cap, dtype=torch.int32, pin_memory=True) if world > 1 else None
         h2d = sum(int(qc.nbytes + qo.nbytes + S.nbytes) for _s, _q, qc, qo, _v in jobs)
         d2h = sum(int(v.numel() * 4) for *_x, v in jobs) if world == 1 else world * cap * 4
-        barrier()
-        torch.cuda.synchronize()
-        t0 = time.perf_counter()
-        for _ in range(args.e2e_steps):
+        def e2e_step():
             if world == 1:
                 for s, qs, qc, qo, view in jobs:
                     h.search(qc, qo, dbs[s], S, 10, 2, out=host_out[s], stream=stream)  # H2D + D2H inside
@@ -372,6 +369,13 @@ def run_ours(args):
                 gather()
                 if rank == 0:
                     final_host.copy_(gathered, non_blocking=False)
+
+        e2e_step()  # untimed: first host-output call allocates the library's staging buffer
+        barrier()
+        torch.cuda.synchronize()
+        t0 = time.perf_counter()
+        for _ in range(args.e2e_steps):
+            e2e_step()
         torch.cuda.synchronize()
         dt = time.perf_counter() - t0
         dtt = torch.tensor([dt], dtype=torch.float64, device=cdev)

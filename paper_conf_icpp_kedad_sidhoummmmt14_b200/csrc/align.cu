@@ -28,6 +28,8 @@
 //             2 = H == E_ij, 3 = otherwise (F_ij)
 //   bit 2     E_ij == H_{i,j-1} - Gs - Ge   (gap opened here, Eq. (3))
 //   bit 3     F_ij == H_{i-1,j} - Gs - Ge   (gap opened here, Eq. (4))
+#include <algorithm>
+
 #include "sw_internal.h"
 #include "sw_device.cuh"
 
@@ -45,31 +47,45 @@ __device__ __forceinline__ bool better(const Best& a, const Best& b) {
 }
 }  // namespace
 
+// TW = warps per pair ("team"): 8 chains the strips of tall queries across the
+// CTA; 1 lets every warp take its own pair (queries of one 256-row strip, where
+// a whole CTA per pair would leave 7 warps idle).
+template <int TW>
+__device__ __forceinline__ void team_sync() {
+  if constexpr (TW == 1) __syncwarp();
+  else if constexpr (TW == ALIGN_WARPS) __syncthreads();
+  else asm volatile("bar.sync %0, %1;" :: "r"(1 + int(threadIdx.x >> 5) / TW), "r"(TW * 32) : "memory");
+}
+
+template <int TW>
 __global__ void __launch_bounds__(ALIGN_WARPS * 32) align_fwd_kernel(AlignArgs a) {
   constexpr int R = ALIGN_R;
-  constexpr int W = ALIGN_WARPS;
+  constexpr int W = TW;  // warps chained on one pair
   constexpr int SW = 33;
   __shared__ int32_t sm[SW * SW];
-  __shared__ int s_prog[W];
-  __shared__ Best s_best[W];
-  __shared__ int s_item;
+  __shared__ int s_prog_all[ALIGN_WARPS];
+  __shared__ Best s_best_all[ALIGN_WARPS];
+  __shared__ int s_item_all[ALIGN_WARPS / TW];
   for (int x = threadIdx.x; x < SW * SW; x += blockDim.x) {
     const int r = x / SW, c = x % SW;
     sm[x] = (r < a.alpha && c < a.alpha) ? int(a.matrix[r * a.alpha + c]) : int(PAD_S);
   }
-  const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
+  const int lane = threadIdx.x & 31, team = (threadIdx.x >> 5) / TW, warp = (threadIdx.x >> 5) % TW;
   const bool lead = lane == 0, tail = lane == 31;
-  int2* __restrict__ links = a.links + (size_t)blockIdx.x * W * a.bcap;
+  int* s_prog = s_prog_all + team * TW;
+  Best* s_best = s_best_all + team * TW;
+  int2* __restrict__ links = a.links + ((size_t)blockIdx.x * ALIGN_WARPS + size_t(team) * TW) * a.bcap;
   const int pad = a.alpha;
   const int nGe = -a.Ge, nGsGe = -(a.Gs + a.Ge);
   const uint32_t padw = uint32_t(pad) * 0x01010101u;
+  __syncthreads();  // matrix staged
   for (;;) {
-    __syncthreads();
-    if (threadIdx.x == 0) s_item = atomicAdd(a.work_counter, 1);
-    if (threadIdx.x < W) s_prog[threadIdx.x] = -1;
-    __syncthreads();
-    const int item = s_item;
-    if (item >= a.n_items) break;
+    team_sync<TW>();
+    if (warp == 0 && lane == 0) s_item_all[team] = atomicAdd(a.work_counter, 1);
+    if (warp == 0 && lane < TW) s_prog[lane] = -1;
+    team_sync<TW>();
+    const int item = a.item_begin + s_item_all[team];
+    if (item >= a.item_begin + a.n_launch) break;
     const AlignItem it = a.items[item];
     const PairRec pr = a.pairs[it.pair];
     const uint8_t* qc = a.qcodes + a.qoff[it.q];
@@ -192,8 +208,8 @@ __global__ void __launch_bounds__(ALIGN_WARPS * 32) align_fwd_kernel(AlignArgs a
       if (better(o, acc)) acc = o;
     }
     if (lane == 0) s_best[warp] = acc;
-    __syncthreads();
-    if (threadIdx.x == 0) {
+    team_sync<TW>();
+    if (warp == 0 && lane == 0) {
       Best b = s_best[0];
       for (int w = 1; w < W; ++w)
         if (better(s_best[w], b)) b = s_best[w];
@@ -272,12 +288,29 @@ __global__ void align_tb_kernel(AlignArgs a) {
   out[5] = overflow ? -n : n;
 }
 
-cudaError_t launch_align(int grid, const AlignArgs& a, cudaStream_t st) {
-  if (a.n_items <= 0) return cudaSuccess;
-  align_fwd_kernel<<<grid, ALIGN_WARPS * 32, 0, st>>>(a);
-  cudaError_t e = cudaGetLastError();
-  if (e != cudaSuccess) return e;
-  align_tb_kernel<<<(a.n_items + 127) / 128, 128, 0, st>>>(a);
+// items [0, n_single) have one strip (warp per pair), [n_single, n_items) are
+// taller (CTA per pair); counters[0..1] zeroed by the caller.
+cudaError_t launch_align(int grid, int n_single, const AlignArgs& a0, int* counters, cudaStream_t st) {
+  if (a0.n_items <= 0) return cudaSuccess;
+  AlignArgs a = a0;
+  if (n_single > 0) {
+    a.item_begin = 0;
+    a.n_launch = n_single;
+    a.work_counter = counters;
+    const int g = std::max(1, std::min(grid, (n_single + ALIGN_WARPS - 1) / ALIGN_WARPS));
+    align_fwd_kernel<1><<<g, ALIGN_WARPS * 32, 0, st>>>(a);
+    cudaError_t e = cudaGetLastError();
+    if (e != cudaSuccess) return e;
+  }
+  if (a0.n_items > n_single) {
+    a.item_begin = n_single;
+    a.n_launch = a0.n_items - n_single;
+    a.work_counter = counters + 1;
+    align_fwd_kernel<ALIGN_WARPS><<<std::min(grid, a.n_launch), ALIGN_WARPS * 32, 0, st>>>(a);
+    cudaError_t e = cudaGetLastError();
+    if (e != cudaSuccess) return e;
+  }
+  align_tb_kernel<<<(a0.n_items + 127) / 128, 128, 0, st>>>(a0);
   return cudaGetLastError();
 }
 

@@ -1001,7 +1001,20 @@ int32_t sw_align(sw_handle_t h, const uint8_t* q_codes, const int64_t* q_offsets
     if (qtot) SW_CK(cudaMemcpyAsync(h->a_qcodes.p, qbase, size_t(qtot), cudaMemcpyHostToDevice, st));
     SW_CK(cudaMemcpyAsync(h->a_qoff.p, qoff0.data(), qoff0.size() * sizeof(int64_t), cudaMemcpyHostToDevice, st));
     SW_CK(cudaMemcpyAsync(h->a_matrix.p, matrix, size_t(alpha * alpha), cudaMemcpyHostToDevice, st));
-    SW_CK(h->a_counter.ensure(sizeof(int)));
+    SW_CK(h->a_counter.ensure(2 * sizeof(int)));
+    // single-strip pairs (query <= 256 rows: one warp each) first, then the taller ones
+    {
+      std::vector<size_t> ord(items.size());
+      std::iota(ord.begin(), ord.end(), size_t(0));
+      std::stable_partition(ord.begin(), ord.end(), [&](size_t x) { return qlen[size_t(items[x].q)] <= 32 * ALIGN_R; });
+      std::vector<AlignItem> it2;
+      std::vector<int32_t> ip2;
+      std::vector<int64_t> w2;
+      for (size_t x : ord) { it2.push_back(items[x]); ip2.push_back(item_pair[x]); w2.push_back(words[x]); }
+      items.swap(it2);
+      item_pair.swap(ip2);
+      words.swap(w2);
+    }
     const int64_t budget = h->opt_align_ws_mb * (int64_t(1) << 20) / 4;  // words
     std::vector<uint32_t> hops;
     std::vector<int32_t> hout;
@@ -1032,7 +1045,9 @@ int32_t sw_align(sw_handle_t h, const uint8_t* q_codes, const int64_t* q_offsets
       SW_CK(h->a_links.ensure(size_t(grid) * size_t(per_cta)));
       SW_CK(cudaMemcpyAsync(h->a_items.p, items.data() + b0, size_t(nb) * sizeof(AlignItem), cudaMemcpyHostToDevice,
                             st));
-      SW_CK(cudaMemsetAsync(h->a_counter.p, 0, sizeof(int), st));
+      SW_CK(cudaMemsetAsync(h->a_counter.p, 0, 2 * sizeof(int), st));
+      int n_single = 0;
+      for (size_t x = b0; x < b1; ++x) n_single += qlen[size_t(items[x].q)] <= 32 * ALIGN_R ? 1 : 0;
       AlignArgs a{};
       a.qcodes = h->a_qcodes.as<uint8_t>();
       a.qoff = h->a_qoff.as<int64_t>();
@@ -1051,7 +1066,7 @@ int32_t sw_align(sw_handle_t h, const uint8_t* q_codes, const int64_t* q_offsets
       a.out = h->a_out.as<int32_t>();
       a.Gs = gap_open;
       a.Ge = gap_extend;
-      SW_CK(launch_align(grid, a, st));
+      SW_CK(launch_align(grid, n_single, a, h->a_counter.as<int>(), st));
       hout.resize(size_t(nb) * 6);
       hops.resize(size_t(std::max<int64_t>(ow, 1)));
       SW_CK(cudaMemcpyAsync(hout.data(), h->a_out.p, hout.size() * sizeof(int32_t), cudaMemcpyDeviceToHost, st));

@@ -205,7 +205,8 @@ struct AlignArgs {
   const int8_t* matrix;      // alpha x alpha
   int alpha;
   const AlignItem* items;    // this batch
-  int n_items;
+  int n_items;               // items of the batch (traceback launch)
+  int item_begin, n_launch;  // items [item_begin, item_begin + n_launch) of one forward launch
   int* work_counter;         // zeroed
   int2* links;               // per-CTA warp link rows, [gridDim][ALIGN_WARPS][bcap]
   int bcap;
@@ -223,6 +224,6 @@ void cpu_search_avx2(const uint8_t* qcodes, const int64_t* qoff, int32_t nq, con
 
 constexpr int ALIGN_WARPS = 8;
 constexpr int ALIGN_R = 8;   // rows per lane = codes per trace word
-cudaError_t launch_align(int grid, const AlignArgs& a, cudaStream_t st);
+cudaError_t launch_align(int grid, int n_single, const AlignArgs& a, int* counters, cudaStream_t st);
 
 }  // namespace swdual

@@ -343,7 +343,7 @@ def run_ours(args):
     alg_bytes = int(n_pass * int(d_lens.sum()) + 4 * Q * N)
     traffic = None
     tpath = os.path.join(ROOT, "profiles", "traffic.json")
-    if os.path.exists(tpath):
+    if os.path.exists(tpath) and args.n_db is None:  # the captured traffic is for the full-size workload
         try:
             t = json.load(open(tpath)).get(args.workload)
             traffic = t.get("traffic_bytes_per_launch") if t else None

@@ -84,8 +84,22 @@ __global__ void __launch_bounds__(ALIGN_WARPS * 32) align_fwd_kernel(AlignArgs a
     if (warp == 0 && lane == 0) s_item_all[team] = atomicAdd(a.work_counter, 1);
     if (warp == 0 && lane < TW) s_prog[lane] = -1;
     team_sync<TW>();
-    const int item = a.item_begin + s_item_all[team];
-    if (item >= a.item_begin + a.n_launch) break;
+    // TW = 8: sub-item x = (pair, CTA c of K) -- tall pairs are split over K = strips/8
+    // CTAs, CTA c taking strips 8c .. 8c+7 (the host sizes K for one round), chained CTA
+    // to CTA through global rows + GPU-scope counters like the re-score kernel.
+    int item, c = 0, K = 1, sub = 0;
+    if constexpr (TW == ALIGN_WARPS) {
+      sub = s_item_all[team];
+      if (sub >= a.n_sub) break;
+      const int2 xm = a.submap[sub];
+      item = xm.x;
+      c = xm.y;
+      K = a.items[item].K;
+    } else {
+      item = a.item_begin + s_item_all[team];
+      if (item >= a.item_begin + a.n_launch) break;
+    }
+    const int sub0 = sub - c;  // this pair's first sub-item: its global rows / counters / partials
     const AlignItem it = a.items[item];
     const PairRec pr = a.pairs[it.pair];
     const uint8_t* qc = a.qcodes + a.qoff[it.q];
@@ -99,16 +113,31 @@ __global__ void __launch_bounds__(ALIGN_WARPS * 32) align_fwd_kernel(AlignArgs a
     const int jw = W - 1 - warp;  // producers on higher warp ids
     Best acc{0, 0x7fffffff, 0x7fffffff};
     for (int r = 0;; ++r) {
-      const int s = W * r + jw;
+      const int s = W * (K * r + c) + jw;
       if (s >= nstrips || L == 0) break;
       const bool rd = s > 0, wr = s + 1 < nstrips;
       Link lk{};
-      const int jl = (jw + W - 1) % W;
-      const int2* rp = links + (size_t)jl * a.bcap + 31;
-      lk.in = &s_prog[jl];
+      const int2* rp;
+      int2* wp;
+      if (jw > 0 || K == 1) {
+        const int jl = (jw + W - 1) % W;
+        rp = links + (size_t)jl * a.bcap + 31;
+        lk.in = &s_prog[jl];
+      } else {  // first warp of a CTA: the strip above is the previous CTA's last
+        const int pc = (c + K - 1) % K;
+        rp = a.grows + (int64_t)(sub0 + pc) * a.bcap + 31;
+        lk.in = a.gflags + sub0 + pc;
+        lk.in_gpu = true;
+      }
       lk.in_base = (s - 1) << 20;
-      int2* wp = links + (size_t)jw * a.bcap;
-      lk.out = &s_prog[jw];
+      if (jw < W - 1 || K == 1) {
+        wp = links + (size_t)jw * a.bcap;
+        lk.out = &s_prog[jw];
+      } else {
+        wp = a.grows + (int64_t)(sub0 + c) * a.bcap;
+        lk.out = a.gflags + sub0 + c;
+        lk.out_gpu = true;
+      }
       lk.out_base = s << 20;
       int qr[R], Hl[R], E[R];
 #pragma unroll
@@ -194,7 +223,10 @@ __global__ void __launch_bounds__(ALIGN_WARPS * 32) align_fwd_kernel(AlignArgs a
           sC = rC;
           if (wr && tail) __stcg(wp + t0 + jj, make_int2(sH, sF));
         }
-        if (wr && tail) st_release_cta(lk.out, lk.out_base + t0 + 4);
+        if (wr && tail) {
+          if (!lk.out_gpu) st_release_cta(lk.out, lk.out_base + t0 + 4);
+          else if (((t0 >> 2) & 3) == 3 || t0 + 4 >= T) st_release_gpu(lk.out, lk.out_base + t0 + 4);
+        }
       }
       if (better(sb, acc)) acc = sb;
     }
@@ -213,7 +245,22 @@ __global__ void __launch_bounds__(ALIGN_WARPS * 32) align_fwd_kernel(AlignArgs a
       Best b = s_best[0];
       for (int w = 1; w < W; ++w)
         if (better(s_best[w], b)) b = s_best[w];
-      a.best[item] = b.v > 0 ? make_int4(b.v, b.i, b.j, 0) : make_int4(0, 0, 0, 0);
+      if (K == 1) {
+        a.best[item] = b.v > 0 ? make_int4(b.v, b.i, b.j, 0) : make_int4(0, 0, 0, 0);
+      } else {  // the last of the K CTAs merges their maxima in the same order
+        a.partial[sub0 + c] = make_int4(b.v, b.j, b.i, 0);
+        __threadfence();
+        if (atomicAdd(a.done + item, 1) == K - 1) {
+          __threadfence();
+          Best m{0, 0x7fffffff, 0x7fffffff};
+          for (int x = 0; x < K; ++x) {
+            const int4 p = __ldcg(a.partial + sub0 + x);
+            const Best o{p.x, p.y, p.z};
+            if (better(o, m)) m = o;
+          }
+          a.best[item] = m.v > 0 ? make_int4(m.v, m.i, m.j, 0) : make_int4(0, 0, 0, 0);
+        }
+      }
     }
   }
 }
@@ -302,11 +349,9 @@ cudaError_t launch_align(int grid, int n_single, const AlignArgs& a0, int* count
     cudaError_t e = cudaGetLastError();
     if (e != cudaSuccess) return e;
   }
-  if (a0.n_items > n_single) {
-    a.item_begin = n_single;
-    a.n_launch = a0.n_items - n_single;
+  if (a0.n_sub > 0) {
     a.work_counter = counters + 1;
-    align_fwd_kernel<ALIGN_WARPS><<<std::min(grid, a.n_launch), ALIGN_WARPS * 32, 0, st>>>(a);
+    align_fwd_kernel<ALIGN_WARPS><<<std::min(grid, a0.n_sub), ALIGN_WARPS * 32, 0, st>>>(a);
     cudaError_t e = cudaGetLastError();
     if (e != cudaSuccess) return e;
   }

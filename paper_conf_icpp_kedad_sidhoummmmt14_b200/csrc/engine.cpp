@@ -111,6 +111,7 @@ struct sw_handle_s {
   int64_t opt_align_ws_mb = 2048;  // sw_align: traceback-code workspace per batch
   // sw_align scratch (separate from sw_search's: a search may still be running on another stream)
   DevBuf a_qcodes, a_qoff, a_matrix, a_items, a_links, a_trace, a_best, a_ops, a_out, a_counter;
+  DevBuf a_submap, a_grows, a_gflags, a_partial, a_done;
   // last-search bookkeeping
   sw_stats_t stats{};
   cudaStream_t last_stream = nullptr;
@@ -1043,11 +1044,34 @@ int32_t sw_align(sw_handle_t h, const uint8_t* q_codes, const int64_t* q_offsets
       const int64_t per_cta = int64_t(ALIGN_WARPS) * bcap * int64_t(sizeof(int2));
       grid = int(std::max<int64_t>(1, std::min<int64_t>(grid, std::max<int64_t>(h->sms, link_budget / per_cta))));
       SW_CK(h->a_links.ensure(size_t(grid) * size_t(per_cta)));
-      SW_CK(cudaMemcpyAsync(h->a_items.p, items.data() + b0, size_t(nb) * sizeof(AlignItem), cudaMemcpyHostToDevice,
-                            st));
       SW_CK(cudaMemsetAsync(h->a_counter.p, 0, 2 * sizeof(int), st));
       int n_single = 0;
       for (size_t x = b0; x < b1; ++x) n_single += qlen[size_t(items[x].q)] <= 32 * ALIGN_R ? 1 : 0;
+      // very tall pairs (> 48 strips, queries > 12k rows): K = strips / 8 CTAs, one round
+      // of 8 strips per CTA, so a CTA only ever waits on CTAs of lower sub-item index
+      // (already running): no circular wait.  Shorter pairs keep one CTA and pipeline
+      // their rounds inside it (measured: splitting config-3 top hits made them 2.6x slower).
+      std::vector<int2> submap;
+      for (size_t x = b0 + size_t(n_single); x < b1; ++x) {
+        const int64_t ns = (qlen[size_t(items[x].q)] + 32 * ALIGN_R - 1) / (32 * ALIGN_R);
+        const int K = ns > 6 * ALIGN_WARPS ? int((ns + ALIGN_WARPS - 1) / ALIGN_WARPS) : 1;
+        items[x].K = K;
+        for (int c = 0; c < K; ++c) submap.push_back(make_int2(int(x - b0), c));
+      }
+      for (size_t x = b0; x < b0 + size_t(n_single); ++x) items[x].K = 1;
+      const int n_sub = int(submap.size());
+      SW_CK(h->a_submap.ensure(std::max<size_t>(submap.size(), 1) * sizeof(int2)));
+      SW_CK(h->a_grows.ensure(std::max<size_t>(submap.size(), 1) * size_t(bcap) * sizeof(int2)));
+      SW_CK(h->a_gflags.ensure(std::max<size_t>(submap.size(), 1) * sizeof(int)));
+      SW_CK(h->a_partial.ensure(std::max<size_t>(submap.size(), 1) * sizeof(int4)));
+      SW_CK(h->a_done.ensure(size_t(nb) * sizeof(int)));
+      if (n_sub) {
+        SW_CK(cudaMemcpyAsync(h->a_submap.p, submap.data(), submap.size() * sizeof(int2), cudaMemcpyHostToDevice, st));
+        SW_CK(cudaMemsetAsync(h->a_gflags.p, 0, submap.size() * sizeof(int), st));
+      }
+      SW_CK(cudaMemsetAsync(h->a_done.p, 0, size_t(nb) * sizeof(int), st));
+      SW_CK(cudaMemcpyAsync(h->a_items.p, items.data() + b0, size_t(nb) * sizeof(AlignItem), cudaMemcpyHostToDevice,
+                            st));
       AlignArgs a{};
       a.qcodes = h->a_qcodes.as<uint8_t>();
       a.qoff = h->a_qoff.as<int64_t>();
@@ -1066,6 +1090,12 @@ int32_t sw_align(sw_handle_t h, const uint8_t* q_codes, const int64_t* q_offsets
       a.out = h->a_out.as<int32_t>();
       a.Gs = gap_open;
       a.Ge = gap_extend;
+      a.submap = h->a_submap.as<int2>();
+      a.n_sub = n_sub;
+      a.grows = h->a_grows.as<int2>();
+      a.gflags = h->a_gflags.as<int>();
+      a.partial = h->a_partial.as<int4>();
+      a.done = h->a_done.as<int>();
       SW_CK(launch_align(grid, n_single, a, h->a_counter.as<int>(), st));
       hout.resize(size_t(nb) * 6);
       hops.resize(size_t(std::max<int64_t>(ow, 1)));

@@ -194,7 +194,7 @@ struct AlignItem {
   int32_t half;              // 0 = low byte (id0), 1 = high byte (id1)
   int32_t n;                 // real DB sequence length
   int32_t ops_cap;           // capacity of the output region
-  int32_t pad_;
+  int32_t K;                 // CTAs the pair is split over (tall queries)
 };
 
 struct AlignArgs {
@@ -206,7 +206,13 @@ struct AlignArgs {
   int alpha;
   const AlignItem* items;    // this batch
   int n_items;               // items of the batch (traceback launch)
-  int item_begin, n_launch;  // items [item_begin, item_begin + n_launch) of one forward launch
+  int item_begin, n_launch;  // single-strip launch: items [item_begin, item_begin + n_launch)
+  const int2* submap;        // tall-pair launch: sub-item -> (item, CTA c of K), a pair's K consecutive
+  int n_sub;
+  int2* grows;               // CTA-to-CTA rows, [n_sub][bcap]
+  int* gflags;               // their progress counters, [n_sub], zeroed
+  int4* partial;             // per sub-item best {v, j, i}
+  int* done;                 // per item finished CTAs, zeroed
   int* work_counter;         // zeroed
   int2* links;               // per-CTA warp link rows, [gridDim][ALIGN_WARPS][bcap]
   int bcap;

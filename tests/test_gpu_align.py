@@ -164,3 +164,19 @@ def test_align_nucleotides_fig1_and_random():
         _check(qc, qo, dc, do, pairs, S.astype(np.int32), gs, ge, 5)
     got = _run(qc, qo, dc, do, [(0, 0)], S, 0, 2, 5)
     assert got[0][0] == 5
+
+
+def test_align_very_tall_query_split_over_ctas():
+    """Queries above 48 strips (12,288 rows) are split over K = strips / 8 CTAs
+    chained through global rows; the K partial end cells merge in (value, j, i)
+    order.  A small alphabet makes equal maxima in different CTAs likely."""
+    rng = np.random.default_rng(31)
+    alpha = 4
+    S = rng.integers(-3, 4, size=(alpha, alpha))
+    ql = [12289, 13000]
+    dl = [180, 7, 640]
+    qc, qo = _seqs(ql, rng, alpha)
+    dc, do = _seqs(dl, rng, alpha)
+    dc[do[2]:do[2] + 500] = qc[qo[1] + 9000:qo[1] + 9500]   # a long diagonal in the lower CTAs
+    pairs = [(q, d) for q in range(len(ql)) for d in range(len(dl))]
+    _check(qc, qo, dc, do, pairs, S, 2, 1, alpha)

@@ -406,6 +406,18 @@ def run_ours(args):
     if rank == 0 and world == 1 and not args.no_cpu_baseline:
         cpu = cpu_baseline(c, args.cpu_baseline_cells)
 
+    # second denominator: the measured register-resident cell-update
+    # microbenchmark at the kernel's occupancy (tools/dpx_microbench.cu, 2 CTAs/SM)
+    micro = None
+    mpath = os.path.join(ROOT, "profiles", "r01_dpx_microbench.jsonl")
+    if os.path.exists(mpath):
+        for ln in open(mpath):
+            try:
+                d = json.loads(ln)
+            except ValueError:
+                continue
+            if d.get("probe") == "gotoh_cellpair_D_max3_R24" and d.get("blocks_per_sm") == 2:
+                micro = float(d["GCUPS"])
     if rank == 0:
         line = {"metric": METRIC, "value": round(value, 2), "unit": "GCUPS", "n_gpus": world, "steps": args.steps,
                 "warmup": args.warmup, "ms_per_step": round(T / args.steps, 3), "higher_is_better": True,
@@ -419,7 +431,11 @@ def run_ours(args):
                              "kernel": "inter_kernel (the persistent scoring launch: long and short pairs), CUDA events around each launch",
                              "peak_basis": f"{n_sm} SMs x {ALU_LANES_PER_SM_CLK} ALU-pipe lanes/clk x {sm_max:.0f} MHz / "
                                            f"{OPS_PER_CELL} ALU lane-ops per cell (minimal s16x2 Gotoh update; "
-                                           f"derived from unit counts + measured pipe attribution)"},
+                                           f"derived from unit counts + measured pipe attribution)",
+                             "microbench_ceiling": micro,
+                             "frac_vs_microbench": round(achieved / micro, 4) if (achieved and micro) else None,
+                             "microbench_basis": "register-resident s16x2 cell update, same 3.5-ALU-op form, 2 CTAs/SM, "
+                                                 "no memory or shuffles (profiles/r01_dpx_microbench.jsonl)"},
                 "cpu_baseline": cpu, "e2e": e2e, "gpu_launches": int(n_launch_step * args.steps),
                 **({"verified_sample": args.verify, "verified": verified} if args.verify else {}),
                 "clocks": clk,

@@ -635,7 +635,10 @@ __global__ void __launch_bounds__(NT) inter_kernel(InterArgs a) {
 
 // ---------------------------------------------------------------------------
 // Instantiation table.
-constexpr int INTER_NT = 256;
+#ifndef SW_INTER_NT
+#define SW_INTER_NT 256
+#endif
+constexpr int INTER_NT = SW_INTER_NT;  // threads per CTA of the scoring kernel
 
 #define SW_INTER_CASES(X)                                                          \
   X(4, 8) X(4, 12) X(4, 16) X(4, 20) X(4, 24) X(4, 28) X(4, 32)                    \

@@ -50,7 +50,10 @@ struct ProfGeom {
   int il;          // 1: unit-interleaved [letter][unit][lane][UB] (long mode); 0: [letter][lane][LB]
 };
 
-constexpr int LONG_R = 16;   // rows per lane of the intra-task (long pair) geometry, G = 32;
+#ifndef SW_LONG_R
+#define SW_LONG_R 16
+#endif
+constexpr int LONG_R = SW_LONG_R;   // rows per lane of the intra-task (long pair) geometry, G = 32;
                              // profile unit-interleaved ([letter][unit][lane][8 B]): dense and
                              // bank-conflict-free (the 16 lanes of an LDS.64 phase hit 16 distinct
                              // 8-byte slots whatever letters they read)

@@ -64,7 +64,8 @@ int32_t sw_init(int32_t device, uint32_t flags, sw_handle_t* out);
  *   out         receives the DB; free with sw_free_db (or sw_free).
  * The inputs are copied; the call returns when the upload is complete.
  * Errors: SW_EINVAL (null pointer, bad offsets, code >= alphabet_size,
- * alphabet_size out of range), SW_ENOMEM, SW_ECUDA.
+ * alphabet_size out of range), SW_ENOMEM, SW_ECUDA, SW_EUNSUPPORTED (a sequence
+ * longer than 2^20 - 128 residues; UniProt's longest has 35,213, L762-764).
  */
 int32_t sw_load_db(sw_handle_t h, const uint8_t* codes, const int64_t* offsets, int64_t n_seqs,
                    int32_t alphabet_size, void* cuda_stream, sw_db_t* out);
@@ -83,7 +84,9 @@ int32_t sw_load_db(sw_handle_t h, const uint8_t* codes, const int64_t* offsets, 
  * synchronizes.  Host `scores`: the call returns after the results are copied.
  * Exactness: scores are exact int32; the int16 DPX path flags any pair whose
  * maximum reaches 32767 - max(matrix) and re-scores it in int32.
- * Errors: SW_EINVAL, SW_ESTATE (db from another handle), SW_ENOMEM, SW_ECUDA.
+ * Errors: SW_EINVAL, SW_ESTATE (db from another handle), SW_ENOMEM, SW_ECUDA,
+ * SW_EUNSUPPORTED (a query longer than 2^19 = 524,288 residues; the longest
+ * UniProt protein, has 35,213).
  * n_queries == 0 or an empty DB is valid and writes nothing.
  */
 int32_t sw_search(sw_handle_t h, const uint8_t* q_codes, const int64_t* q_offsets, int32_t n_queries,
@@ -118,8 +121,8 @@ int32_t sw_search(sw_handle_t h, const uint8_t* q_codes, const int64_t* q_offset
  * batched under the "align_workspace_mb" option), then one thread per pair
  * walks it.
  * Errors: SW_EINVAL (bad index, code, gaps, null pointer, a region too small
- * for the path), SW_ESTATE, SW_ENOMEM, SW_ECUDA, SW_EUNSUPPORTED (a sequence
- * longer than 2^20 - 64).
+ * for the path), SW_ESTATE, SW_ENOMEM, SW_ECUDA, SW_EUNSUPPORTED (a DB sequence
+ * longer than 2^20 - 64 or a query longer than 2^19).
  */
 int32_t sw_align(sw_handle_t h, const uint8_t* q_codes, const int64_t* q_offsets, int32_t n_queries, sw_db_t db,
                  const int32_t* pairs, int32_t n_pairs, const int8_t* matrix, int32_t gap_open, int32_t gap_extend,

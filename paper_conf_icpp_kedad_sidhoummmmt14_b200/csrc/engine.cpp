@@ -293,6 +293,9 @@ int32_t sw_load_db(sw_handle_t h, const uint8_t* codes, const int64_t* offsets, 
     } catch (const std::invalid_argument& e) {
       fail(SW_EINVAL, std::string("sw_load_db: ") + e.what());
     }
+    // strip progress counters encode (strip << 20) + column (kernels.cu): columns < 2^20
+    if (P.max_len > (int64_t(1) << 20) - 128)
+      fail(SW_EUNSUPPORTED, "sw_load_db: a sequence is longer than 2^20 - 128 residues");
     db->n_res = P.n_res;
     db->max_len = P.max_len;
     db->n_long = P.n_long;
@@ -781,7 +784,8 @@ int32_t sw_search(sw_handle_t h, const uint8_t* q_codes, const int64_t* q_offset
     for (int i = 0; i < n_queries; ++i) {
       qlen[size_t(i)] = q_offsets[i + 1] - q_offsets[i];
       if (qlen[size_t(i)] < 0) fail(SW_EINVAL, "sw_search: q_offsets not non-decreasing");
-      if (qlen[size_t(i)] > (int64_t(1) << 30)) fail(SW_EUNSUPPORTED, "sw_search: query longer than 2^30");
+      // strip progress counters encode (strip << 20) + column: strips of >= 256 rows, < 2^11 of them
+      if (qlen[size_t(i)] > (int64_t(1) << 19)) fail(SW_EUNSUPPORTED, "sw_search: query longer than 2^19 residues");
       qtot += qlen[size_t(i)];
     }
     if (qtot > 0 && !q_codes) fail(SW_EINVAL, "sw_search: q_codes is NULL");
@@ -952,7 +956,7 @@ int32_t sw_align(sw_handle_t h, const uint8_t* q_codes, const int64_t* q_offsets
     for (int i = 0; i < n_queries; ++i) {
       qlen[size_t(i)] = q_offsets[i + 1] - q_offsets[i];
       if (qlen[size_t(i)] < 0) fail(SW_EINVAL, "sw_align: q_offsets not non-decreasing");
-      if (qlen[size_t(i)] > (int64_t(1) << 30)) fail(SW_EUNSUPPORTED, "sw_align: query longer than 2^30");
+      if (qlen[size_t(i)] > (int64_t(1) << 19)) fail(SW_EUNSUPPORTED, "sw_align: query longer than 2^19 residues");
       qtot += qlen[size_t(i)];
     }
     if (qtot > 0 && !q_codes) fail(SW_EINVAL, "sw_align: q_codes is NULL");

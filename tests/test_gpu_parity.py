@@ -322,3 +322,19 @@ def test_hybrid_cpu_gpu_search():
     assert (plan.pe < 3).any() and (plan.pe == 3).any()
     np.testing.assert_array_equal(got, oracle_scores(qc, qo, c["dcodes"], c["doff"]))
     np.testing.assert_array_equal(got_dp, got)
+
+
+def test_length_limits():
+    """Sequences beyond the kernels' counter encoding are refused, not mis-scored."""
+    sw = _pkg()
+    big = np.zeros((1 << 20), dtype=np.uint8)
+    with sw.Handle(0) as h:
+        with pytest.raises(sw.SWError) as e:
+            h.load_db(big, np.array([0, len(big)], dtype=np.int64))
+        assert e.value.code == sw._lib.SW_EUNSUPPORTED
+        db = h.load_db(big[:100], np.array([0, 100], dtype=np.int64))
+        q = np.zeros((1 << 19) + 1, dtype=np.uint8)
+        with pytest.raises(sw.SWError) as e:
+            h.search(q, np.array([0, len(q)], dtype=np.int64), db, sw.blosum62(), 10, 2,
+                     out=np.zeros((1, 1), dtype=np.int32))
+        assert e.value.code == sw._lib.SW_EUNSUPPORTED

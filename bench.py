@@ -69,6 +69,9 @@ def parse():
     ap.add_argument("--force-geom", default=None, help="G,R of the inter-task kernel (experiments; default auto)")
     ap.add_argument("--verify", type=int, default=0, help="after timing, check N sampled DB sequences "
                     "of the assembled scores against the CPU oracle (rank 0)")
+    ap.add_argument("--gather", default="nccl", choices=["nccl", "fused"],
+                    help="N > 1: all-gather of score blocks (nccl) or fused: every rank's scoring epilogue writes "
+                         "into rank 0's score matrix mapped over NVLink (CUDA IPC), no collective on the data path")
     ap.add_argument("--dist-backend", default="nccl", help="nccl (default); gloo only for functional checks "
                     "of the multi-rank path on a box with fewer GPUs than ranks")
     return ap.parse_args()
@@ -145,6 +148,8 @@ def config_obj(args, c, q_lens, d_lens, n):
             "n_db_seqs": int(len(d_lens)), "db_residues": int(d_lens.sum()),
             "matrix": "BLOSUM62", "gap_open": 10, "gap_extend": 2,
             "shards": n, "placement": "dual-approximation (query, shard) tasks",
+            **({"gather": "fused epilogue into rank 0's matrix over CUDA IPC / NVLink" if args.gather == "fused"
+                else "NCCL all-gather of score blocks"} if n > 1 else {}),
             "l2": "inputs larger than L2: 205 MB packed DB > 126 MB L2, streamed once per query per step"
             if args.workload in ("c2", "c3", "t5hom", "t5het") and args.n_db is None else "small workload"}
 
@@ -267,10 +272,26 @@ def run_ours(args):
         fg, fr = (int(x) for x in args.force_geom.split(","))
         h.set_option("force_G", fg)
         h.set_option("force_R", fr)
+    fused = args.gather == "fused" and world > 1
+    full_dev = None
+    if fused:  # rank 0 owns scores[Q][N]; the other ranks map it (CUDA IPC; peer access over NVLink)
+        from torch.multiprocessing.reductions import reduce_tensor
+        if rank == 0:
+            full_dev = torch.zeros((Q, N), dtype=torch.int32, device=dev)
+            obj = [reduce_tensor(full_dev)]
+        else:
+            obj = [None]
+        pg.broadcast_object_list(obj, src=0)
+        if rank != 0:
+            fn, fargs = obj[0]
+            full_dev = fn(*fargs)
     dbs = {}
     for s, _qs in blocks:
         sc, so = swdist.subset(c["dcodes"], c["doff"], shards[s])
-        dbs[s] = h.load_db(sc, so, alphabet_size=24)
+        if fused:  # scores land in columns shards[s] of rank 0's rows of N
+            dbs[s] = h.load_db(sc, so, alphabet_size=24, out_index=shards[s], out_n=N)
+        else:
+            dbs[s] = h.load_db(sc, so, alphabet_size=24)
     # per block: query subset (host), device output view into one flat buffer
     sizes = [swdist.flat_size(plan, r) for r in range(world)]
     cap = max(max(sizes), 1)
@@ -279,6 +300,16 @@ def run_ours(args):
     jobs = []
     pos = 0
     for s, qs in blocks:
+        if fused:  # one search per run of consecutive queries: rows a..b of the shared matrix
+            runs, a0 = [], 0
+            for i in range(1, len(qs) + 1):
+                if i == len(qs) or qs[i] != qs[i - 1] + 1:
+                    runs.append(qs[a0:i])
+                    a0 = i
+            for run in runs:
+                qc, qo = swdist.subset(c["qcodes"], c["qoff"], run)
+                jobs.append((s, run, qc, qo, full_dev[run[0]:run[-1] + 1]))
+            continue
         qc, qo = swdist.subset(c["qcodes"], c["qoff"], qs)
         n = len(shards[s])
         view = flat[pos:pos + len(qs) * n].view(len(qs), n)
@@ -297,7 +328,7 @@ def run_ours(args):
     def step():
         for s, qs, qc, qo, view in jobs:
             h.search(qc, qo, dbs[s], S, 10, 2, out=view, stream=stream)
-        if world > 1:
+        if world > 1 and not fused:
             gather()
 
     for _ in range(args.warmup):
@@ -365,13 +396,21 @@ def run_ours(args):
         host_out = {}
         for s, qs, qc, qo, view in jobs:
             host_out[s] = torch.empty(tuple(view.shape), dtype=torch.int32, pin_memory=True).numpy()
-        final_host = torch.empty(world * cap, dtype=torch.int32, pin_memory=True) if world > 1 else None
+        final_host = (torch.empty(Q * N if fused else world * cap, dtype=torch.int32, pin_memory=True)
+                      if world > 1 else None)
         h2d = sum(int(qc.nbytes + qo.nbytes + S.nbytes) for _s, _q, qc, qo, _v in jobs)
-        d2h = sum(int(v.numel() * 4) for *_x, v in jobs) if world == 1 else world * cap * 4
+        d2h = sum(int(v.numel() * 4) for *_x, v in jobs) if world == 1 else (Q * N * 4 if fused else world * cap * 4)
         def e2e_step():
             if world == 1:
                 for s, qs, qc, qo, view in jobs:
                     h.search(qc, qo, dbs[s], S, 10, 2, out=host_out[s], stream=stream)  # H2D + D2H inside
+            elif fused:
+                for s, qs, qc, qo, view in jobs:
+                    h.search(qc, qo, dbs[s], S, 10, 2, out=view, stream=stream)      # epilogue writes rank 0's rows
+                torch.cuda.synchronize()
+                barrier()
+                if rank == 0:
+                    final_host.copy_(full_dev.view(-1), non_blocking=False)
             else:
                 for s, qs, qc, qo, view in jobs:
                     h.search(qc, qo, dbs[s], S, 10, 2, out=view, stream=stream)      # H2D of queries inside
@@ -395,12 +434,18 @@ def run_ours(args):
 
     verified = None
     if args.verify > 0:
-        if world > 1:
+        if world > 1 and not fused:
             gather()
             torch.cuda.synchronize()
+        if fused:
+            torch.cuda.synchronize()
+            barrier()
         if rank == 0:
-            g = (gathered if world > 1 else flat).cpu().numpy().reshape(world, -1)
-            full = swdist.assemble(plan, Q, N, [g[r] for r in range(world)])
+            if fused:
+                full = full_dev.cpu().numpy()
+            else:
+                g = (gathered if world > 1 else flat).cpu().numpy().reshape(world, -1)
+                full = swdist.assemble(plan, Q, N, [g[r] for r in range(world)])
             import oracle
             from oracle.blosum62 import blosum62 as ob62
             rng = np.random.default_rng(5)

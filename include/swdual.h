@@ -71,6 +71,21 @@ int32_t sw_load_db(sw_handle_t h, const uint8_t* codes, const int64_t* offsets, 
                    int32_t alphabet_size, void* cuda_stream, sw_db_t* out);
 
 /*
+ * sw_load_db with an output mapping (the scoring epilogue writes a
+ * shard's scores straight into the full matrix, e.g. rank 0's buffer mapped into
+ * this process over NVLink with CUDA IPC, so no gather collective follows).
+ *   out_index   host, int64[n_seqs]: distinct output columns in [0, out_n).
+ *   out_n       columns of the output rows (>= n_seqs).
+ * sw_search on such a DB treats `scores` as int32[n_queries][out_n] (device or
+ * peer-mapped memory only) and writes only this DB's columns, leaving the
+ * others untouched.  sw_align keeps the caller's local DB indices.
+ * Errors: as sw_load_db; SW_EINVAL for a bad mapping.
+ */
+int32_t sw_load_db_mapped(sw_handle_t h, const uint8_t* codes, const int64_t* offsets, int64_t n_seqs,
+                          int32_t alphabet_size, const int64_t* out_index, int64_t out_n, void* cuda_stream,
+                          sw_db_t* out);
+
+/*
  * Score every (query, database sequence) pair.
  *   q_codes, q_offsets   host, queries in the same layout as sw_load_db
  *                        (int64 q_offsets[n_queries + 1]); codes < alphabet.

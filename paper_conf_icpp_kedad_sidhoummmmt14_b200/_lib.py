@@ -16,7 +16,7 @@ SW_FLAG_TIMING = 1
 
 EXPORTS = ["sw_init", "sw_load_db", "sw_search", "sw_free_db", "sw_free", "sw_last_error",
            "sw_db_info", "sw_last_stats", "sw_set_option", "sw_encode_ascii", "sw_schedule_dual", "sw_align",
-           "sw_encode_nucleotide", "sw_search_cpu", "sw_schedule_dual_dp"]
+           "sw_encode_nucleotide", "sw_search_cpu", "sw_schedule_dual_dp", "sw_load_db_mapped"]
 
 
 class SWError(RuntimeError):
@@ -75,6 +75,8 @@ def lib() -> ctypes.CDLL:
     L.sw_schedule_dual.argtypes = [I64, V, V, I32, I32, V, P(ctypes.c_double), P(ctypes.c_double)]
     L.sw_encode_nucleotide.restype = I32
     L.sw_encode_nucleotide.argtypes = [ctypes.c_char_p, I64, V]
+    L.sw_load_db_mapped.restype = I32
+    L.sw_load_db_mapped.argtypes = [V, V, V, I64, I32, V, I64, V, P(V)]
     L.sw_schedule_dual_dp.restype = I32
     L.sw_schedule_dual_dp.argtypes = [I64, V, V, I32, I32, V, P(ctypes.c_double), P(ctypes.c_double)]
     L.sw_search_cpu.restype = I32

@@ -72,14 +72,24 @@ class Handle:
     def set_option(self, key: str, value: int) -> None:
         check(lib().sw_set_option(self.ptr, key.encode(), int(value)), self.ptr)
 
-    def load_db(self, codes, offsets, alphabet_size: int = 24, stream=None) -> Database:
+    def load_db(self, codes, offsets, alphabet_size: int = 24, stream=None, out_index=None,
+                out_n: int | None = None) -> Database:
+        """sw_load_db, or sw_load_db_mapped when out_index is given: the scores of
+        sequence d then land in column out_index[d] of rows of out_n columns."""
         codes = _host(codes, np.uint8)
         offsets = _host(offsets, np.int64)
         n = len(offsets) - 1
         out = ctypes.c_void_p()
-        check(lib().sw_load_db(self.ptr, _vp(codes) if codes.size else None, _vp(offsets), n, int(alphabet_size),
-                               _stream_ptr(stream), ctypes.byref(out)), self.ptr)
+        if out_index is None:
+            check(lib().sw_load_db(self.ptr, _vp(codes) if codes.size else None, _vp(offsets), n, int(alphabet_size),
+                                   _stream_ptr(stream), ctypes.byref(out)), self.ptr)
+        else:
+            oi = _host(out_index, np.int64)
+            check(lib().sw_load_db_mapped(self.ptr, _vp(codes) if codes.size else None, _vp(offsets), n,
+                                          int(alphabet_size), _vp(oi) if oi.size else None, int(out_n),
+                                          _stream_ptr(stream), ctypes.byref(out)), self.ptr)
         db = Database(self, out, n)
+        db.out_n = n if out_index is None else int(out_n)
         db.seq_lens = np.diff(offsets)
         self._dbs.append(db)
         return db
@@ -96,7 +106,7 @@ class Handle:
         q_offsets = _host(q_offsets, np.int64)
         matrix = _host(matrix, np.int8)
         nq = len(q_offsets) - 1
-        N = db.n_seqs
+        N = getattr(db, "out_n", db.n_seqs)
         if out is None:
             if torch is not None and torch.cuda.is_available():
                 out = torch.empty((nq, N), dtype=torch.int32, device=f"cuda:{self.device}")

@@ -136,6 +136,12 @@ struct sw_db_s {
   DevBuf dlofs;
   DevBuf stream, dpairs;
   std::vector<int64_t> seq_loc;  // caller index -> 2 * pair + half (-1: empty); built on first sw_align
+  // output mapping (sw_load_db_mapped): scores of sequence d land in column out_index[d] of
+  // rows of out_n columns -- e.g. a rank's shard writing into rank 0's full matrix
+  int64_t out_n = 0;
+  bool mapped = false;
+  DevBuf dzero_cols;             // mapped: output columns of empty sequences (zeroed per search)
+  int64_t n_zero_cols = 0;
 };
 
 static int32_t set_err(sw_handle_s* h, int32_t code, const std::string& m) {
@@ -286,6 +292,7 @@ int32_t sw_load_db(sw_handle_t h, const uint8_t* codes, const int64_t* offsets, 
     db = new sw_db_s();
     db->h = h;
     db->n_seqs = n_seqs;
+    db->out_n = n_seqs;
     db->alpha = alphabet_size;
     Packed P;
     try {
@@ -340,6 +347,54 @@ int32_t sw_load_db(sw_handle_t h, const uint8_t* codes, const int64_t* offsets, 
   h->dbs.push_back(db);
   *out = db;
   return SW_OK;
+}
+
+int32_t sw_load_db_mapped(sw_handle_t h, const uint8_t* codes, const int64_t* offsets, int64_t n_seqs,
+                          int32_t alphabet_size, const int64_t* out_index, int64_t out_n, void* cuda_stream,
+                          sw_db_t* out) {
+  if (!h) return set_err(nullptr, SW_EINVAL, "sw_load_db_mapped: handle is NULL");
+  if (!out) return set_err(h, SW_EINVAL, "sw_load_db_mapped: out is NULL");
+  if (n_seqs > 0 && !out_index) return set_err(h, SW_EINVAL, "sw_load_db_mapped: out_index is NULL");
+  if (out_n < n_seqs) return set_err(h, SW_EINVAL, "sw_load_db_mapped: out_n < n_seqs");
+  {  // distinct columns in [0, out_n)
+    std::vector<uint8_t> seen(size_t(std::max<int64_t>(out_n, 1)), 0);
+    for (int64_t d = 0; d < n_seqs; ++d) {
+      const int64_t x = out_index[d];
+      if (x < 0 || x >= out_n || seen[size_t(x)]) return set_err(h, SW_EINVAL, "sw_load_db_mapped: out_index not distinct in [0, out_n)");
+      seen[size_t(x)] = 1;
+    }
+  }
+  int32_t rc = sw_load_db(h, codes, offsets, n_seqs, alphabet_size, cuda_stream, out);
+  if (rc != SW_OK) return rc;
+  sw_db_s* db = *out;
+  rc = guarded(h, [&] {
+    cudaStream_t st = reinterpret_cast<cudaStream_t>(cuda_stream);
+    // device pair table with output columns instead of caller indices (the host copy keeps them)
+    std::vector<PairRec> dp(db->pairs);
+    for (auto& r : dp) {
+      r.id0 = int32_t(out_index[r.id0]);
+      if (r.id1 >= 0) r.id1 = int32_t(out_index[r.id1]);
+    }
+    if (out_n > (int64_t(1) << 31) - 1) fail(SW_EUNSUPPORTED, "sw_load_db_mapped: out_n >= 2^31");
+    if (!dp.empty())
+      SW_CK(cudaMemcpyAsync(db->dpairs.p, dp.data(), dp.size() * sizeof(PairRec), cudaMemcpyHostToDevice, st));
+    std::vector<int64_t> zc;
+    for (int64_t d = 0; d < n_seqs; ++d)
+      if (db->seq_len[size_t(d)] == 0) zc.push_back(out_index[d]);
+    db->n_zero_cols = int64_t(zc.size());
+    if (!zc.empty()) {
+      SW_CK(db->dzero_cols.ensure(zc.size() * sizeof(int64_t)));
+      SW_CK(cudaMemcpyAsync(db->dzero_cols.p, zc.data(), zc.size() * sizeof(int64_t), cudaMemcpyHostToDevice, st));
+    }
+    db->out_n = out_n;
+    db->mapped = true;
+    SW_CK(cudaStreamSynchronize(st));
+  });
+  if (rc != SW_OK) {
+    sw_free_db(db);
+    *out = nullptr;
+  }
+  return rc;
 }
 
 int32_t sw_db_info(sw_db_t db, sw_db_info_t* out) {
@@ -540,7 +595,7 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
     QueryDesc& d = desc[k];
     d.prof = nullptr;
     d.prof_long = prof + off_l[k];
-    d.scores = c.dscores + int64_t(qi) * db->n_seqs;
+    d.scores = c.dscores + int64_t(qi) * db->out_n;
     d.n_strips = 0;
     d.n_strips_long = gl[k].n_strips;
     d.qidx = qi;
@@ -587,7 +642,7 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
     d.mode = sl.mode;
     d.n_strips = strips_s[j];
     d.qidx0 = order[size_t(sl.A[0])];
-    d.scores0 = c.dscores + int64_t(d.qidx0) * db->n_seqs;
+    d.scores0 = c.dscores + int64_t(d.qidx0) * db->out_n;
     d.qidx1 = -1;
     d.scores1 = nullptr;
     d.sinfo = nullptr;
@@ -737,7 +792,7 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
   a.bcap = bcap;
   a.work_counter = h->counters.as<int>();
   a.scores_all = c.dscores;
-  a.n_seqs = db->n_seqs;
+  a.n_seqs = db->out_n;
   a.thr = c.thr;
   a.ovf = c.ovf;
   a.ovf_count = c.ovf_count;
@@ -803,9 +858,11 @@ int32_t sw_search(sw_handle_t h, const uint8_t* q_codes, const int64_t* q_offset
     if (cudaPointerGetAttributes(&pa, scores) == cudaSuccess)
       dev_scores = (pa.type == cudaMemoryTypeDevice || pa.type == cudaMemoryTypeManaged);
     cudaGetLastError();
-    const int64_t N = db->n_seqs;
+    const int64_t N = db->out_n;  // row stride of the output (n_seqs unless the DB is mapped)
     const size_t out_bytes = size_t(n_queries) * size_t(N) * sizeof(int32_t);
     int32_t* dscores = scores;
+    if (db->mapped && !dev_scores)
+      fail(SW_EINVAL, "sw_search: a DB loaded with sw_load_db_mapped needs device (or peer-mapped) scores");
     if (!dev_scores) {
       SW_CK(h->scores_tmp.ensure(out_bytes));
       dscores = h->scores_tmp.as<int32_t>();
@@ -824,8 +881,13 @@ int32_t sw_search(sw_handle_t h, const uint8_t* q_codes, const int64_t* q_offset
     if (qtot) SW_CK(cudaMemcpyAsync(h->qcodes.p, qbase, size_t(qtot), cudaMemcpyHostToDevice, st));
     SW_CK(cudaMemcpyAsync(h->qoff.p, qoff0.data(), qoff0.size() * sizeof(int64_t), cudaMemcpyHostToDevice, st));
     SW_CK(cudaMemcpyAsync(h->matrix.p, matrix, size_t(alpha * alpha), cudaMemcpyHostToDevice, st));
-    SW_CK(cudaMemsetAsync(dscores, 0, out_bytes, st));
     int launches = 0;
+    if (!db->mapped) {
+      SW_CK(cudaMemsetAsync(dscores, 0, out_bytes, st));
+    } else if (db->n_zero_cols > 0) {  // only this DB's columns: other ranks write the rest
+      SW_CK(launch_zero_columns(dscores, N, n_queries, db->dzero_cols.as<int64_t>(), db->n_zero_cols, st));
+      ++launches;
+    }
     // overflow list capacity: a pair can only be flagged if min(m, n) * S_max >= thr
     int64_t ovf_cap = 0;
     if (smax > 0) {

@@ -16,6 +16,7 @@
 //   * the int8 query profile of the current strip sits in shared memory;
 //   * CTAs are persistent and take chunks of NT/G pairs from an atomic counter,
 //     pairs sorted longest first.
+#include <algorithm>
 #include <cstdio>
 #include "sw_internal.h"
 #include "sw_device.cuh"
@@ -856,6 +857,22 @@ __global__ void __launch_bounds__(RESCORE_WARPS * 32) rescore_kernel(RescoreArgs
 
 cudaError_t launch_rescore(int grid, const RescoreArgs& a, cudaStream_t st) {
   rescore_kernel<<<grid, RESCORE_WARPS * 32, 0, st>>>(a);  // persistent; K CTAs per flagged pair
+  return cudaGetLastError();
+}
+
+// Mapped DBs (sw_load_db_mapped): the empty sequences' output columns are zeroed
+// individually, because the rest of each row belongs to other shards.
+__global__ void zero_columns_kernel(int32_t* scores, int64_t stride, int nq, const int64_t* cols, int64_t ncols) {
+  const int64_t n = int64_t(nq) * ncols;
+  for (int64_t x = blockIdx.x * int64_t(blockDim.x) + threadIdx.x; x < n; x += int64_t(gridDim.x) * blockDim.x)
+    scores[(x / ncols) * stride + cols[x % ncols]] = 0;
+}
+
+cudaError_t launch_zero_columns(int32_t* scores, int64_t stride, int nq, const int64_t* cols, int64_t ncols,
+                                cudaStream_t st) {
+  const int64_t n = int64_t(nq) * ncols;
+  if (n <= 0) return cudaSuccess;
+  zero_columns_kernel<<<int(std::min<int64_t>((n + 255) / 256, 1024)), 256, 0, st>>>(scores, stride, nq, cols, ncols);
   return cudaGetLastError();
 }
 

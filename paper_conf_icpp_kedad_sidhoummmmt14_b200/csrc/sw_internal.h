@@ -182,6 +182,9 @@ cudaError_t launch_inter(int G, int R, int NT, int grid, int smem_bytes, const I
 bool inter_config_supported(int G, int R);
 int inter_block_threads();  // NT of the scoring kernel (its long items use NT/32 chained warps)
 cudaError_t launch_rescore(int grid, const RescoreArgs& a, cudaStream_t st);
+// scores[q * stride + cols[c]] = 0 for every query q < nq and column c < ncols
+cudaError_t launch_zero_columns(int32_t* scores, int64_t stride, int nq, const int64_t* cols, int64_t ncols,
+                                cudaStream_t st);
 constexpr int RESCORE_WARPS = 8;
 constexpr int RESCORE_R = 8;
 

@@ -338,3 +338,40 @@ def test_length_limits():
             h.search(q, np.array([0, len(q)], dtype=np.int64), db, sw.blosum62(), 10, 2,
                      out=np.zeros((1, 1), dtype=np.int32))
         assert e.value.code == sw._lib.SW_EUNSUPPORTED
+
+
+def test_mapped_db_writes_into_shared_matrix():
+    """sw_load_db_mapped (SURVEY 8(e) fusion): shards loaded with their caller
+    columns write straight into one [Q][N] device matrix, leaving the other
+    shards' columns untouched (sentinels survive until their own shard runs)."""
+    import torch
+    sw = _pkg()
+    from paper_conf_icpp_kedad_sidhoummmmt14_b200 import dist
+    c = swgen.make_config("c1", n_db=700)
+    dc, do = c["dcodes"].copy(), c["doff"].copy()
+    lens = np.diff(do)
+    lens[5] = 0                                   # an empty sequence: its column must be zeroed
+    do = np.zeros(len(lens) + 1, dtype=np.int64)
+    np.cumsum(lens, out=do[1:])
+    dc = np.concatenate([c["dcodes"][c["doff"][i]:c["doff"][i] + lens[i]] for i in range(len(lens))])
+    qc, qo = swgen.make_queries(21, [300, 144, 700])
+    N = len(lens)
+    shards = dist.shard_cut(do, 3)
+    with sw.Handle(0) as h:
+        full = torch.full((3, N), -7, dtype=torch.int32, device="cuda")
+        dbs = [h.load_db(*dist.subset(dc, do, idx), out_index=idx, out_n=N) for idx in shards]
+        h.search(qc, qo, dbs[0], sw.blosum62(), 10, 2, out=full)
+        torch.cuda.synchronize()
+        part = full.cpu().numpy()
+        others = np.setdiff1d(np.arange(N), shards[0])
+        assert (part[:, others] == -7).all()
+        for db in dbs[1:]:
+            h.search(qc[:0], qo[:1], db, sw.blosum62(), 10, 2, out=full[:0])   # no queries: writes nothing
+        h.search(qc[qo[1]:], qo[1:] - qo[1], dbs[1], sw.blosum62(), 10, 2, out=full[1:])   # rows 1..2 only
+        h.search(qc, qo, dbs[2], sw.blosum62(), 10, 2, out=full)
+        h.search(qc[:qo[1]], qo[:2], dbs[1], sw.blosum62(), 10, 2, out=full[:1])          # row 0
+        torch.cuda.synchronize()
+        got = full.cpu().numpy()
+        with pytest.raises(sw.SWError):   # host output is refused for a mapped DB
+            h.search(qc, qo, dbs[0], sw.blosum62(), 10, 2, out=np.zeros((3, N), dtype=np.int32))
+    np.testing.assert_array_equal(got, oracle_scores(qc, qo, dc, do))

@@ -189,8 +189,16 @@ static ProfGeom make_geom(int G, int R, int m, int alpha, bool long_mode = false
 // (row padding to whole strips, wavefront fill of G-1 columns per pair and
 // strip, a per-step overhead amortised over R rows, a register-pressure
 // penalty for the largest R).
+// Small searches (few cells) are bound by their critical path -- one lane group
+// sweeping the tallest query's strips over the longest short pair -- rather than by
+// throughput.  Per wavefront step a lane spends about 18.4 cycles per row plus ~99
+// of shuffles / loads (fit on config 1: G,R = 4,24 / 8,24 / 16,16 / 16,8 / 32,8 /
+// 32,12 measured 1.11 / 0.60 / 0.39 / 0.45 / 0.26 / 0.38 ms, model within 12 %).
+constexpr double SMALL_SEARCH_CELLS = 2e10;   // below this, minimise max(throughput, critical path)
+constexpr double CELLS_PER_CYCLE = 3500.0;    // whole-GPU throughput of the short-pair mode (config 3)
+
 static void choose_geom(const sw_handle_s* h, const std::vector<std::pair<int, int>>& slots, double Lavg, int& G,
-                        int& R) {
+                        int& R, double Lmax = 0.0, double real_cells = 1e300) {
   if (h->opt_G > 0 && h->opt_R > 0) {
     G = int(h->opt_G);
     R = int(h->opt_R);
@@ -211,6 +219,14 @@ static void choose_geom(const sw_handle_s* h, const std::vector<std::pair<int, i
         // mode 1 (query pair) sweeps every DB sequence once for two queries, without the PRMT
         const double cols = mode == 1 ? 2.0 * (Lavg + g) * (5.5 / 6.5) : (Lavg + g);
         cost += rows * cols * per_cell * (strips > 1 ? 1.02 : 1.0);
+      }
+      if (real_cells < SMALL_SEARCH_CELLS && Lmax > 0) {  // in cycles: max(throughput, critical path)
+        int mmax = 0;
+        for (auto [m, mode] : slots) mmax = std::max(mmax, m);
+        const int strips = std::max(1, (mmax + g * r - 1) / (g * r));
+        const int V = (r % 8 == 0) ? 2 : 1;
+        const double cp = double(strips) * (Lmax + double(g * V)) * (18.4 * r + 99.0);
+        cost = std::max(cost / CELLS_PER_CYCLE, cp);
       }
       if (cost < best) { best = cost; G = g; R = r; }
     }
@@ -459,7 +475,10 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
   }
   const int nshort_db = np - db->n_long;  // (only for the geometry cost model)
   int G = 4, R = 24;
-  choose_geom(h, slot_m, nshort_db > 0 ? db->sum_short_len / nshort_db : 1.0, G, R);
+  double qsum = 0;
+  for (int m : ms) qsum += m;
+  choose_geom(h, slot_m, nshort_db > 0 ? db->sum_short_len / nshort_db : 1.0, G, R, double(db->max_short),
+              qsum * double(db->n_res));
   if (!inter_config_supported(G, R)) fail(SW_EUNSUPPORTED, "no kernel for this geometry");
   const int NT = inter_block_threads(), NG = NT / G, W = NT / 32;
   const int LB2 = (((R / 4) | 1) * 16);

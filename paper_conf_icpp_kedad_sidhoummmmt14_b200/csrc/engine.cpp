@@ -219,6 +219,10 @@ static void choose_geom(const sw_handle_s* h, const std::vector<std::pair<int, i
         // mode 1 (query pair) sweeps every DB sequence once for two queries, without the PRMT
         const double cols = mode == 1 ? 2.0 * (Lavg + g) * (5.5 / 6.5) : (Lavg + g);
         cost += rows * cols * per_cell * (strips > 1 ? 1.02 : 1.0);
+        // single-query mode: each extra strip pass also costs ~6.7 cell-equivalents per
+        // column (boundary-row round trip + pass setup; fit on config 2, where 3 passes
+        // of G = 8 beat 6 passes of G = 4 by 1.9 % at equal row padding)
+        if (mode == 0 && strips > 1) cost += 6.7 * double(strips) * Lavg;
       }
       if (real_cells < SMALL_SEARCH_CELLS && Lmax > 0) {  // in cycles: max(throughput, critical path)
         int mmax = 0;

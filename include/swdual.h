@@ -206,6 +206,10 @@ int32_t sw_last_stats(sw_handle_t h, sw_stats_t* out);
  *                         pair > 3000 when such pairs hold most of the residues)
  *   "pack_long"           1: pack several long pairs per CTA when a query has
  *                         fewer intra-task strips than warps (default 0)
+ *   "resident_strips"     1: a multi-strip query slot whose whole profile fits
+ *                         in the CTA's shared-memory share keeps every strip
+ *                         resident (no per-pass reload), 0: one strip at a
+ *                         time (default 0: measured neutral)
  *   "timing"              1/0, same as SW_FLAG_TIMING
  *   "timing_accumulate"   1: short_ms/long_ms of sw_last_stats sum every search
  *                         since the last "timing_reset" (0: the last search only)

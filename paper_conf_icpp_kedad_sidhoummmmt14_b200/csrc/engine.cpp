@@ -107,6 +107,8 @@ struct sw_handle_s {
   int64_t opt_query_pairs = 1;  // pair queries two per register for the short pairs
   int64_t opt_pack_queries = 1; // mode-1 slots: fill the shorter half with further queries (strip-aligned)
   int64_t opt_bank_copy = 1;    // query-pair profile: second smem copy shifted by 64 B for odd lane groups
+  int64_t opt_resident = 0;     // multi-strip slots whose whole profile fits: all strips resident in smem
+                                // (same-box A/B: neutral within 0.2% on C1-C3, Table V; kept off)
   int64_t opt_pack_long = 0;    // 1: several long pairs per CTA item when a query has fewer strips than warps
   int64_t opt_align_ws_mb = 2048;  // sw_align: traceback-code workspace per batch
   // sw_align scratch (separate from sw_search's: a search may still be running on another stream)
@@ -286,6 +288,8 @@ int32_t sw_set_option(sw_handle_t h, const char* key, int64_t value) {
     h->opt_pack_queries = value;
   } else if (k == "bank_copy") {
     h->opt_bank_copy = value;
+  } else if (k == "resident_strips") {
+    h->opt_resident = value;
   } else if (k == "query_pairs") {
     h->opt_query_pairs = value;
   } else if (k == "timing_accumulate") {
@@ -669,6 +673,7 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
     d.qidx1 = -1;
     d.scores1 = nullptr;
     d.sinfo = nullptr;
+    d.res_stride = 0;
     uint8_t* vA = nullptr;
     uint8_t* vB = nullptr;
     if (sl.mode == 1) {
@@ -748,11 +753,6 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
   SW_CK(h->imap.ensure(std::max<size_t>(imap.size(), 1) * sizeof(int2)));
   if (!imap.empty())
     SW_CK(cudaMemcpyAsync(h->imap.p, imap.data(), imap.size() * sizeof(int2), cudaMemcpyHostToDevice, c.st));
-  SW_CK(h->qdesc.ensure(desc.size() * sizeof(QueryDesc) + sdesc.size() * sizeof(SlotDesc) + 16));
-  QueryDesc* d_desc = h->qdesc.as<QueryDesc>();
-  SlotDesc* d_slots = reinterpret_cast<SlotDesc*>(d_desc + desc.size());
-  SW_CK(cudaMemcpyAsync(d_desc, desc.data(), desc.size() * sizeof(QueryDesc), cudaMemcpyHostToDevice, c.st));
-  SW_CK(cudaMemcpyAsync(d_slots, sdesc.data(), sdesc.size() * sizeof(SlotDesc), cudaMemcpyHostToDevice, c.st));
   int max_strips = 1;
   for (int n : strips_s) max_strips = std::max(max_strips, n);
   const ProfGeom l0 = gl[0];
@@ -762,10 +762,45 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
   const int cstride2 = SB2 + (ncopy2 > 1 ? 128 / ncopy2 : 0);
   const int sprof_bytes = std::max((ncopy0 - 1) * cstride0 + g1.SB, (ncopy2 - 1) * cstride2 + SB2);
   // an item is either short or long: the long-mode slots reuse the same bytes
-  const int smem = SW_SMEM_UNION ? std::max(sprof_bytes, nlong_max > 0 ? W * l0.SB : 0)
+  int smem = SW_SMEM_UNION ? std::max(sprof_bytes, nlong_max > 0 ? W * l0.SB : 0)
                                  : sprof_bytes + (nlong_max > 0 ? W * l0.SB : 0);
-  const int occ = inter_max_ctas_per_sm(G, R, NT, smem);
+  int occ = inter_max_ctas_per_sm(G, R, NT, smem);
   if (occ <= 0) fail(SW_ECUDA, "inter kernel does not fit on an SM");
+  // Resident strips: a multi-strip slot whose strips (with their bank copies) all
+  // fit in the per-CTA shared-memory share of the current occupancy keeps them
+  // resident, so its items load the profile once instead of once per strip pass
+  // (two CTA barriers per pass saved).  Kept only if the occupancy does not drop.
+  if (h->opt_resident) {
+    const int long_part = nlong_max > 0 ? W * l0.SB : 0;
+    const int stride0 = (((ncopy0 - 1) * cstride0 + g1.SB) + 127) / 128 * 128;
+    const int stride2 = (((ncopy2 - 1) * cstride2 + SB2) + 127) / 128 * 128;
+    const int cap = 233472 / occ - 2048 - (SW_SMEM_UNION ? 0 : long_part);
+    int res_bytes = sprof_bytes;
+    bool any = false;
+    for (size_t j2 = 0; j2 < sdesc.size(); ++j2) {
+      SlotDesc& d = sdesc[j2];
+      const int stride = d.mode == 1 ? stride2 : stride0;
+      const int64_t need = int64_t(d.n_strips) * stride;
+      if (d.n_items > 0 && d.n_strips > 1 && need <= cap) {
+        d.res_stride = stride;
+        res_bytes = std::max(res_bytes, int(need));
+        any = true;
+      }
+    }
+    if (any) {
+      const int smem_r = SW_SMEM_UNION ? std::max(res_bytes, long_part) : res_bytes + long_part;
+      if (inter_max_ctas_per_sm(G, R, NT, smem_r) >= occ) {
+        smem = smem_r;
+      } else {
+        for (auto& d : sdesc) d.res_stride = 0;
+      }
+    }
+  }
+  SW_CK(h->qdesc.ensure(desc.size() * sizeof(QueryDesc) + sdesc.size() * sizeof(SlotDesc) + 16));
+  QueryDesc* d_desc = h->qdesc.as<QueryDesc>();
+  SlotDesc* d_slots = reinterpret_cast<SlotDesc*>(d_desc + desc.size());
+  SW_CK(cudaMemcpyAsync(d_desc, desc.data(), desc.size() * sizeof(QueryDesc), cudaMemcpyHostToDevice, c.st));
+  SW_CK(cudaMemcpyAsync(d_slots, sdesc.data(), sdesc.size() * sizeof(SlotDesc), cudaMemcpyHostToDevice, c.st));
   const int64_t n_items = long_items + item;
   if (n_items >= (int64_t(1) << 31)) fail(SW_EUNSUPPORTED, "too many work items");
   const int grid = int(std::max<int64_t>(1, std::min<int64_t>(n_items, int64_t(occ) * h->sms)));

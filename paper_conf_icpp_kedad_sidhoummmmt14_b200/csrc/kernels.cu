@@ -567,15 +567,22 @@ __global__ void __launch_bounds__(NT) inter_kernel(InterArgs a) {
       uint32_t best = 0;
       const int SBx = q2 ? a.SB2 : a.SB;
       const int ncp = q2 ? a.ncopy[1] : a.ncopy[0], csx = q2 ? a.cstride[1] : a.cstride[0];
-      const uint8_t* gprof = sprof + (g & (ncp - 1)) * csx;  // this group's bank-spread copy
+      const int rs = d.res_stride;  // > 0: every strip of the slot resident (loaded once per slot)
       for (int s = 0; s < d.n_strips; ++s) {
-        const int want = (sl << 16) | s;
+        const int want = rs ? ((sl << 16) | 0xffff) : ((sl << 16) | s);
         if (want != loaded) {
           __syncthreads();
-          for (int cp = 0; cp < ncp; ++cp) copy_strip(sprof + cp * csx, d.prof + (size_t)s * SBx, SBx);
+          if (rs) {
+            for (int s2 = 0; s2 < d.n_strips; ++s2)
+              for (int cp = 0; cp < ncp; ++cp)
+                copy_strip(sprof + s2 * rs + cp * csx, d.prof + (size_t)s2 * SBx, SBx);
+          } else {
+            for (int cp = 0; cp < ncp; ++cp) copy_strip(sprof + cp * csx, d.prof + (size_t)s * SBx, SBx);
+          }
           __syncthreads();
           loaded = want;
         }
+        const uint8_t* gprof = sprof + (rs ? s * rs : 0) + (g & (ncp - 1)) * csx;  // this group's bank-spread copy
         if (q2) {
           const StripInfo si = d.sinfo[s];
           const bool rd = s > 0 && si.keep != 0;

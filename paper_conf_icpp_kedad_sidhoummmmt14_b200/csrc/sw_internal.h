@@ -107,7 +107,7 @@ struct SlotDesc {
   int item_begin;            // first short work item of this slot
   int n_items;               // short work items of this slot
   int pair_begin;            // short pairs of this slot: [pair_begin, pair_end)
-  int pad_;
+  int res_stride;            // > 0: all strips resident in smem, strip s at s * res_stride (bytes)
 };
 
 struct InterArgs {

@@ -261,6 +261,21 @@ def test_query_packing(pack, thr):
     np.testing.assert_array_equal(got, oracle_scores(qc, qo, dc, do))
 
 
+@pytest.mark.parametrize("resident", [0, 1])
+@pytest.mark.parametrize("pairs", [0, 1])
+def test_resident_strip_profiles(resident, pairs):
+    """Multi-strip slots whose whole profile fits in shared memory keep every
+    strip resident (loaded once per slot); taller ones stream a strip per pass.
+    One search mixes both (2..6-strip queries and a 190-strip one at 32-row
+    strips), in the query-pair and single-query modes."""
+    rng = np.random.default_rng(61 + 2 * resident + pairs)
+    dc, do = _seqs(list(rng.integers(1, 400, size=140)) + [0, 1, 2, 5], rng)
+    qc, qo = _seqs([6077, 150, 64, 65, 33, 190, 31], rng)
+    opts = {"resident_strips": resident, "query_pairs": pairs, "force_G": 4, "force_R": 8}
+    got = gpu_scores(qc, qo, dc, do, opts=opts)
+    np.testing.assert_array_equal(got, oracle_scores(qc, qo, dc, do))
+
+
 @pytest.mark.parametrize("name", ["t5hom", "t5het"])
 def test_table5_query_sets_sampled(name):
     """PAPER.md Table V query sets (40 homogeneous 4,500-5,000 aa / heterogeneous

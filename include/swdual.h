@@ -206,6 +206,9 @@ int32_t sw_last_stats(sw_handle_t h, sw_stats_t* out);
  *                         pair > 3000 when such pairs hold most of the residues)
  *   "pack_long"           1: pack several long pairs per CTA when a query has
  *                         fewer intra-task strips than warps (default 0)
+ *   "bank_skew"           1: single-query profile copies one per lane group of
+ *                         a shared-memory phase at searched bank skews
+ *                         (conflict-free; default 1), 0: the linear layout
  *   "resident_strips"     1: a multi-strip query slot whose whole profile fits
  *                         in the CTA's shared-memory share keeps every strip
  *                         resident (no per-pass reload), 0: one strip at a

@@ -107,6 +107,7 @@ struct sw_handle_s {
   int64_t opt_query_pairs = 1;  // pair queries two per register for the short pairs
   int64_t opt_pack_queries = 1; // mode-1 slots: fill the shorter half with further queries (strip-aligned)
   int64_t opt_bank_copy = 1;    // query-pair profile: second smem copy shifted by 64 B for odd lane groups
+  int64_t opt_bank_skew = 1;    // mode-0 profile copies: per-copy bank skew (mode0_copies)
   int64_t opt_resident = 0;     // multi-strip slots whose whole profile fits: all strips resident in smem
                                 // (same-box A/B: neutral within 0.2% on C1-C3, Table V; kept off)
   int64_t opt_pack_long = 0;    // 1: several long pairs per CTA item when a query has fewer strips than warps
@@ -167,6 +168,54 @@ static int32_t guarded(sw_handle_s* h, F&& f) {
 }
 
 // ----------------------------------------------------------------------------
+// Bank-spread copies of the mode-0 (single-query) strip profile.  Lane k of a
+// group loads its rows at copy + letter * LS + k * LB (+ the row unit, equal for
+// all lanes), LS a multiple of 128 B, so only the copy decides which banks the
+// lane groups of one shared-memory phase hit.  The width of that load is 8 B
+// only when a sub-lane's rows are whole 8-row units (R = 16, 32), else 4 B, so a
+// phase holds 128 / width / G groups.  With 2 to 4 such groups, each copy gets
+// a per-copy skew (multiple of 4 B, exhaustive search) minimising the worst bank
+// load of the phase -- conflict-free for every geometry; the previous linear
+// layout (copy c at c * (SB + 128 / ncopy), sized for 8-byte loads) left 2-way
+// conflicts at R = 8, 24 with G = 8, 16.  Otherwise the linear layout stays.
+struct Mode0Copies { int ncopy, cstride; uint32_t skew; int bytes; };
+static Mode0Copies mode0_copies(int G, int R, int LB, int SB, bool on, bool skewed) {
+  Mode0Copies c{1, SB, 0u, SB};
+  if (!on) return c;
+  const int N = (R % 8 == 0) ? R / 2 : R;               // rows per sub-lane
+  const int w = (R % 8 == 0 && N % 8 == 0) ? 8 : 4;     // bytes per lane per profile load
+  const int gpp = std::max(1, (128 / w) / G);           // lane groups per phase
+  if (!skewed || gpp > 4 || gpp < 2) {                  // linear layout (previous rule)
+    c.ncopy = std::max(1, (128 / (R % 8 == 0 ? 8 : 4)) / G);
+    c.cstride = SB + (c.ncopy > 1 ? 128 / c.ncopy : 0);
+    c.bytes = (c.ncopy - 1) * c.cstride + SB;
+    return c;
+  }
+  c.ncopy = gpp;
+  c.cstride = (SB + 127) / 128 * 128 + 128;
+  // exhaustive over the (up to 3) free skews, lexicographic; stops at conflict-free
+  auto worst_of = [&](const int* sk) {
+    int cnt[32] = {0}, wmax = 0;
+    for (int q = 0; q < c.ncopy; ++q)
+      for (int k = 0; k < G; ++k)
+        for (int b = 0; b < w; b += 4) wmax = std::max(wmax, ++cnt[((sk[q] + k * LB + b) / 4) % 32]);
+    return wmax;
+  };
+  int sk[4] = {0, 0, 0, 0}, best_sk[4] = {0, 0, 0, 0}, best = 1 << 30;
+  const int n1 = c.ncopy > 1 ? 32 : 1, n2 = c.ncopy > 2 ? 32 : 1, n3 = c.ncopy > 3 ? 32 : 1;
+  for (int i1 = 0; i1 < n1 && best > 1; ++i1)
+    for (int i2 = 0; i2 < n2 && best > 1; ++i2)
+      for (int i3 = 0; i3 < n3 && best > 1; ++i3) {
+        sk[1] = 4 * i1; sk[2] = 4 * i2; sk[3] = 4 * i3;
+        const int v = worst_of(sk);
+        if (v < best) { best = v; std::copy(sk, sk + 4, best_sk); }
+      }
+  std::copy(best_sk, best_sk + 4, sk);
+  for (int cp = 0; cp < c.ncopy; ++cp) c.skew |= uint32_t(sk[cp] / 4) << (8 * cp);
+  c.bytes = (c.ncopy - 1) * c.cstride + sk[c.ncopy - 1] + SB;
+  return c;
+}
+
 // geometry of the inter-task kernel for a query of m rows and a launch whose
 // pairs average Lavg columns
 // long = true: the intra-task (G = 32) unit-interleaved layout, LB = the unit
@@ -288,6 +337,8 @@ int32_t sw_set_option(sw_handle_t h, const char* key, int64_t value) {
     h->opt_pack_queries = value;
   } else if (k == "bank_copy") {
     h->opt_bank_copy = value;
+  } else if (k == "bank_skew") {
+    h->opt_bank_skew = value;
   } else if (k == "resident_strips") {
     h->opt_resident = value;
   } else if (k == "query_pairs") {
@@ -500,7 +551,6 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
   const int SB2 = (((alpha + 1) * LS2 + 15) / 16) * 16;
   // copies: lanes of one phase (128 B / unit) divided by the group width
   const int ncopy2 = bank_copy ? std::max(1, (128 / 16) / G) : 1;
-  const int ncopy0 = bank_copy ? std::max(1, (128 / (R % 8 == 0 ? 8 : 4)) / G) : 1;
   // Per slot, pairs [0, nlong) go to the intra-task (long) mode: a short item
   // (one lane group, every strip of its query in turn) must not run much longer
   // than an average lane group's share of the whole launch, or it becomes the
@@ -758,12 +808,13 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
   const ProfGeom l0 = gl[0];
   // copy c of a strip sits at c * cstride; cstride = SB + 128 / ncopy (SB is a
   // multiple of 128 when copies are used)
-  const int cstride0 = g1.SB + (ncopy0 > 1 ? 128 / ncopy0 : 0);
+  const Mode0Copies mc0 = mode0_copies(G, R, g1.LB, g1.SB, bank_copy, h->opt_bank_skew != 0);
+  const int ncopy0 = mc0.ncopy, cstride0 = mc0.cstride;
   const int cstride2 = SB2 + (ncopy2 > 1 ? 128 / ncopy2 : 0);
-  const int sprof_bytes = std::max((ncopy0 - 1) * cstride0 + g1.SB, (ncopy2 - 1) * cstride2 + SB2);
+  const int sprof_bytes = std::max(mc0.bytes, (ncopy2 - 1) * cstride2 + SB2);
   // an item is either short or long: the long-mode slots reuse the same bytes
   int smem = SW_SMEM_UNION ? std::max(sprof_bytes, nlong_max > 0 ? W * l0.SB : 0)
-                                 : sprof_bytes + (nlong_max > 0 ? W * l0.SB : 0);
+                                 : sprof_bytes + 128 + (nlong_max > 0 ? W * l0.SB : 0);
   int occ = inter_max_ctas_per_sm(G, R, NT, smem);
   if (occ <= 0) fail(SW_ECUDA, "inter kernel does not fit on an SM");
   // Resident strips: a multi-strip slot whose strips (with their bank copies) all
@@ -772,7 +823,7 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
   // (two CTA barriers per pass saved).  Kept only if the occupancy does not drop.
   if (h->opt_resident) {
     const int long_part = nlong_max > 0 ? W * l0.SB : 0;
-    const int stride0 = (((ncopy0 - 1) * cstride0 + g1.SB) + 127) / 128 * 128;
+    const int stride0 = (mc0.bytes + 127) / 128 * 128;
     const int stride2 = (((ncopy2 - 1) * cstride2 + SB2) + 127) / 128 * 128;
     const int cap = 233472 / occ - 2048 - (SW_SMEM_UNION ? 0 : long_part);
     int res_bytes = sprof_bytes;
@@ -828,6 +879,7 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
   a.ncopy[1] = ncopy2;
   a.cstride[0] = cstride0;
   a.cstride[1] = cstride2;
+  a.cskew0 = mc0.skew;
   a.LS2 = LS2;
   a.LB2 = LB2;
   a.SB = g1.SB;

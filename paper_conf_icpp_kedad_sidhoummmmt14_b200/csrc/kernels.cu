@@ -123,8 +123,20 @@ cudaError_t launch_build_profile_q2(const uint8_t* qa, int ma, const uint8_t* qb
 // ---------------------------------------------------------------------------
 __device__ __forceinline__ void copy_strip(uint8_t* dst, const uint8_t* __restrict__ src, int bytes) {
   const uint4* s = reinterpret_cast<const uint4*>(src);
-  uint4* d = reinterpret_cast<uint4*>(dst);
-  for (int i = threadIdx.x; i < bytes / 16; i += blockDim.x) d[i] = __ldg(s + i);
+  if ((reinterpret_cast<uintptr_t>(dst) & 15) == 0) {
+    uint4* d = reinterpret_cast<uint4*>(dst);
+    for (int i = threadIdx.x; i < bytes / 16; i += blockDim.x) d[i] = __ldg(s + i);
+  } else {  // bank-skewed copy (4-byte aligned)
+    uint32_t* d = reinterpret_cast<uint32_t*>(dst);
+    for (int i = threadIdx.x; i < bytes / 16; i += blockDim.x) {
+      const uint4 v = __ldg(s + i);
+      d[4 * i] = v.x; d[4 * i + 1] = v.y; d[4 * i + 2] = v.z; d[4 * i + 3] = v.w;
+    }
+  }
+}
+// byte offset of bank-spread copy cp of the short strip profile
+__device__ __forceinline__ int copy_off(int cp, int csx, uint32_t skew) {
+  return cp * csx + 4 * int((skew >> (8 * cp)) & 0xffu);
 }
 
 // DB codes of the current pair: every strip pass of an item re-reads them, so
@@ -377,7 +389,7 @@ __global__ void __launch_bounds__(NT) inter_kernel(InterArgs a) {
   extern __shared__ __align__(16) uint8_t smem[];
   // An item is either short or long, so the two uses share shared memory:
   uint8_t* sprof = smem;                         // short mode: the strip profile (bank-spread copies)
-  uint8_t* lprof = smem + (SW_SMEM_UNION ? 0 : max(a.cstride[0] * (a.ncopy[0] - 1) + a.SB,
+  uint8_t* lprof = smem + (SW_SMEM_UNION ? 0 : max(a.cstride[0] * (a.ncopy[0] - 1) + 128 + a.SB,
                                                     a.cstride[1] * (a.ncopy[1] - 1) + a.SB2));  // long mode: one a.SBL slot per warp
   __shared__ int s_item;
   __shared__ int s_prog[NT / 32];
@@ -567,6 +579,7 @@ __global__ void __launch_bounds__(NT) inter_kernel(InterArgs a) {
       uint32_t best = 0;
       const int SBx = q2 ? a.SB2 : a.SB;
       const int ncp = q2 ? a.ncopy[1] : a.ncopy[0], csx = q2 ? a.cstride[1] : a.cstride[0];
+      const uint32_t skw = q2 ? 0u : a.cskew0;
       const int rs = d.res_stride;  // > 0: every strip of the slot resident (loaded once per slot)
       for (int s = 0; s < d.n_strips; ++s) {
         const int want = rs ? ((sl << 16) | 0xffff) : ((sl << 16) | s);
@@ -575,14 +588,14 @@ __global__ void __launch_bounds__(NT) inter_kernel(InterArgs a) {
           if (rs) {
             for (int s2 = 0; s2 < d.n_strips; ++s2)
               for (int cp = 0; cp < ncp; ++cp)
-                copy_strip(sprof + s2 * rs + cp * csx, d.prof + (size_t)s2 * SBx, SBx);
+                copy_strip(sprof + s2 * rs + copy_off(cp, csx, skw), d.prof + (size_t)s2 * SBx, SBx);
           } else {
-            for (int cp = 0; cp < ncp; ++cp) copy_strip(sprof + cp * csx, d.prof + (size_t)s * SBx, SBx);
+            for (int cp = 0; cp < ncp; ++cp) copy_strip(sprof + copy_off(cp, csx, skw), d.prof + (size_t)s * SBx, SBx);
           }
           __syncthreads();
           loaded = want;
         }
-        const uint8_t* gprof = sprof + (rs ? s * rs : 0) + (g & (ncp - 1)) * csx;  // this group's bank-spread copy
+        const uint8_t* gprof = sprof + (rs ? s * rs : 0) + copy_off(g & (ncp - 1), csx, skw);  // this group's bank-spread copy
         if (q2) {
           const StripInfo si = d.sinfo[s];
           const bool rd = s > 0 && si.keep != 0;

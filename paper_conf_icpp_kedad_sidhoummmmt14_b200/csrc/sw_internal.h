@@ -124,6 +124,9 @@ struct InterArgs {
   // 128/ncopy modulo 128, so the groups of one shared-memory phase (random
   // letters each) hit disjoint banks.  Index 0: mode 0, index 1: mode 1.
   int ncopy[2], cstride[2];
+  // per-copy bank skew of the mode-0 copies: copy c sits at c * cstride[0] +
+  // 4 * ((cskew0 >> 8c) & 0xff) (0 for the linear layout; mode 1 is always linear)
+  uint32_t cskew0;
   int SBL, LSL, LBL;         // long geometry (32 lanes x LONG_R rows)
   int n_long_items;          // sum over queries of n_long * n_super
   uint2* links;              // [gridDim][NT/32][lcap] strip-to-strip rows inside a CTA (long items)

@@ -261,6 +261,20 @@ def test_query_packing(pack, thr):
     np.testing.assert_array_equal(got, oracle_scores(qc, qo, dc, do))
 
 
+@pytest.mark.parametrize("skew", [0, 1])
+@pytest.mark.parametrize("G,R", [(8, 24), (8, 8), (16, 24), (16, 8), (8, 12), (4, 16), (8, 16)])
+def test_single_query_profile_copies(G, R, skew):
+    """Single-query mode (two DB sequences per register) with the bank-skewed
+    profile copies (option bank_skew, one copy per lane group of a shared-memory
+    phase at a searched 4-byte skew) and the linear layout; multi-strip queries."""
+    rng = np.random.default_rng(71 + G * 3 + R + skew)
+    dc, do = _seqs(list(rng.integers(1, 350, size=120)) + [0, 1, 3], rng)
+    qc, qo = _seqs([3 * G * R + 7, G * R, 17], rng)
+    opts = {"bank_skew": skew, "query_pairs": 0, "force_G": G, "force_R": R}
+    got = gpu_scores(qc, qo, dc, do, opts=opts)
+    np.testing.assert_array_equal(got, oracle_scores(qc, qo, dc, do))
+
+
 @pytest.mark.parametrize("resident", [0, 1])
 @pytest.mark.parametrize("pairs", [0, 1])
 def test_resident_strip_profiles(resident, pairs):

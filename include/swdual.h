@@ -209,6 +209,10 @@ int32_t sw_last_stats(sw_handle_t h, sw_stats_t* out);
  *   "bank_skew"           1: single-query profile copies one per lane group of
  *                         a shared-memory phase at searched bank skews
  *                         (conflict-free; default 1), 0: the linear layout
+ *   "wide_profile"        1: single-query slots use 32-bit profile rows and
+ *                         build each cell pair's scores with one IMAD instead
+ *                         of a PRMT (separate kernel; default 0: measured
+ *                         neutral)
  *   "resident_strips"     1: a multi-strip query slot whose whole profile fits
  *                         in the CTA's shared-memory share keeps every strip
  *                         resident (no per-pass reload), 0: one strip at a

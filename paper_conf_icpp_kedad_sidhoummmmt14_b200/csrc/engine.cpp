@@ -108,6 +108,7 @@ struct sw_handle_s {
   int64_t opt_pack_queries = 1; // mode-1 slots: fill the shorter half with further queries (strip-aligned)
   int64_t opt_bank_copy = 1;    // query-pair profile: second smem copy shifted by 64 B for odd lane groups
   int64_t opt_bank_skew = 1;    // mode-0 profile copies: per-copy bank skew (mode0_copies)
+  int64_t opt_wide0 = 0;        // single-query slots: 32-bit profile, pair build by IMAD instead of PRMT
   int64_t opt_resident = 0;     // multi-strip slots whose whole profile fits: all strips resident in smem
                                 // (same-box A/B: neutral within 0.2% on C1-C3, Table V; kept off)
   int64_t opt_pack_long = 0;    // 1: several long pairs per CTA item when a query has fewer strips than warps
@@ -339,6 +340,8 @@ int32_t sw_set_option(sw_handle_t h, const char* key, int64_t value) {
     h->opt_bank_copy = value;
   } else if (k == "bank_skew") {
     h->opt_bank_skew = value;
+  } else if (k == "wide_profile") {
+    h->opt_wide0 = value;
   } else if (k == "resident_strips") {
     h->opt_resident = value;
   } else if (k == "query_pairs") {
@@ -643,13 +646,14 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
     total += qnlong[k] > 0 ? size_t(gl.back().n_strips) * gl.back().SB : 0;
   }
   const ProfGeom g1 = make_geom(G, R, 1, alpha, false, bank_copy);  // SB / LS / LB of the mode-0 profile
+  const bool wide0 = h->opt_wide0 != 0 && inter_wide_supported(G, R);  // mode-0 slots use the 32-bit profile (two sub-lanes only)
   std::vector<size_t> off_s;
   std::vector<int> strips_s;
   for (auto& sl : slots) {
     const int n = sl.strips;
     strips_s.push_back(n);
     off_s.push_back(total);
-    if (sl.nlong < np) total += size_t(n) * (sl.mode == 1 ? SB2 : g1.SB);
+    if (sl.nlong < np) total += size_t(n) * ((sl.mode == 1 || wide0) ? SB2 : g1.SB);
   }
   SW_CK(h->prof.ensure(total + 16));
   uint8_t* prof = h->prof.as<uint8_t>();
@@ -724,6 +728,7 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
     d.scores1 = nullptr;
     d.sinfo = nullptr;
     d.res_stride = 0;
+    d.wide = (sl.mode == 0 && wide0) ? 1 : 0;
     uint8_t* vA = nullptr;
     uint8_t* vB = nullptr;
     if (sl.mode == 1) {
@@ -762,6 +767,10 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
         SW_CK(launch_build_profile_q2(vA, rows, vB, rows, dmat, alpha, G, R, LB2, LS2, d.n_strips, SB2,
                                       prof + off_s[j], c.st));
         cells_computed += 2.0 * (2.0 * sumS) * double(d.n_strips) * G * R;  // every sequence, 2 queries
+      } else if (d.wide) {  // low half S[q_i][a], high half 0 (mb < 0)
+        SW_CK(launch_build_profile_q2(qptr(sl.A[0]), ms[size_t(sl.A[0])], nullptr, -1, dmat, alpha, G, R, LB2, LS2,
+                                      d.n_strips, SB2, prof + off_s[j], c.st));
+        cells_computed += 2.0 * sumS * double(d.n_strips) * G * R;
       } else {
         ProfGeom gq = g1;
         gq.n_strips = d.n_strips;
@@ -815,7 +824,7 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
   // an item is either short or long: the long-mode slots reuse the same bytes
   int smem = SW_SMEM_UNION ? std::max(sprof_bytes, nlong_max > 0 ? W * l0.SB : 0)
                                  : sprof_bytes + 128 + (nlong_max > 0 ? W * l0.SB : 0);
-  int occ = inter_max_ctas_per_sm(G, R, NT, smem);
+  int occ = inter_max_ctas_per_sm(G, R, NT, smem, wide0);
   if (occ <= 0) fail(SW_ECUDA, "inter kernel does not fit on an SM");
   // Resident strips: a multi-strip slot whose strips (with their bank copies) all
   // fit in the per-CTA shared-memory share of the current occupancy keeps them
@@ -830,7 +839,7 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
     bool any = false;
     for (size_t j2 = 0; j2 < sdesc.size(); ++j2) {
       SlotDesc& d = sdesc[j2];
-      const int stride = d.mode == 1 ? stride2 : stride0;
+      const int stride = (d.mode == 1 || d.wide) ? stride2 : stride0;
       const int64_t need = int64_t(d.n_strips) * stride;
       if (d.n_items > 0 && d.n_strips > 1 && need <= cap) {
         d.res_stride = stride;
@@ -840,7 +849,7 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
     }
     if (any) {
       const int smem_r = SW_SMEM_UNION ? std::max(res_bytes, long_part) : res_bytes + long_part;
-      if (inter_max_ctas_per_sm(G, R, NT, smem_r) >= occ) {
+      if (inter_max_ctas_per_sm(G, R, NT, smem_r, wide0) >= occ) {
         smem = smem_r;
       } else {
         for (auto& d : sdesc) d.res_stride = 0;
@@ -880,6 +889,7 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
   a.cstride[0] = cstride0;
   a.cstride[1] = cstride2;
   a.cskew0 = mc0.skew;
+  a.wmul = 65536u;
   a.LS2 = LS2;
   a.LB2 = LB2;
   a.SB = g1.SB;
@@ -915,7 +925,7 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
     h->event_kind[h->n_events_used - 1] = 0;
     SW_CK(cudaEventRecord(ev->first, c.st));
   }
-  SW_CK(launch_inter(G, R, NT, grid, smem, a, c.st));
+  SW_CK(launch_inter(G, R, NT, grid, smem, a, c.st, wide0));
   if (ev) SW_CK(cudaEventRecord(ev->second, c.st));
   ++launches;
   ++h->stats.n_score_launches;

@@ -100,7 +100,7 @@ __global__ void build_profile_q2_kernel(const uint8_t* __restrict__ qa, int ma, 
         // rows past a query, and PAD codes (= alpha) that pad packed queries to whole strips
         const int ca = row < ma ? qa[row] : alpha, cb = row < mb ? qb[row] : alpha;
         const int va = (ca < alpha && a < alpha) ? M[ca * alpha + a] : PAD_SCORE;
-        const int vb = (cb < alpha && a < alpha) ? M[cb * alpha + a] : PAD_SCORE;
+        const int vb = mb < 0 ? 0 : (cb < alpha && a < alpha) ? M[cb * alpha + a] : PAD_SCORE;  // mb < 0: wide mode-0 profile
         v = (uint32_t(va) & 0xffffu) | (uint32_t(vb) << 16);
       }
     }
@@ -206,11 +206,13 @@ struct SubLanes {
   static constexpr int V = (R % 8 == 0) ? 2 : 1;
 };
 
-template <int G, int R, bool LINKED, bool Q2 = false, int US = (Q2 ? 16 : ((R % 8 == 0) ? 8 : 4))>
+template <int G, int R, bool LINKED, bool Q2 = false, int US = (Q2 ? 16 : ((R % 8 == 0) ? 8 : 4)), int PW = 0>
 __device__ __forceinline__ void strip_pass(const uint8_t* sprof, int LS, int LB, const uint16_t* pstream, int L,
                                            int T, int k, bool rd, bool wr, const uint2* __restrict__ rp,
                                            uint2* __restrict__ wp, const Link& lk, uint32_t code_pad2,
-                                           uint32_t nGe, uint32_t nGsGe, uint32_t& best, uint32_t shift = 0) {
+                                           uint32_t nGe, uint32_t nGsGe, uint32_t& best, uint32_t shift = 0,
+                                           uint32_t wmul = 0) {
+  static_assert(!PW || (!Q2 && R % 8 == 0 && US == 16), "wide single-query profile: two sub-lanes, LDS.128 rows");
   constexpr int V = SubLanes<R>::V;
   constexpr int VG = V * G;   // width of the wave in sub-lanes
   constexpr int RH = R / V;   // rows per sub-lane
@@ -319,8 +321,9 @@ __device__ __forceinline__ void strip_pass(const uint8_t* sprof, int LS, int LB,
       }
       if constexpr (V == 2) {
         uint32_t h1 = cH, f1 = cF;
-        if constexpr (SW_DUAL && (Q2 || (SW_DUAL_LONG && LINKED))) {  // measured: +3% for the query-pair mode, -2% with the PRMT (mode 0)
-          gotoh_rows_dual<R, Q2, US>(HA, E, best, hdiag, pa, pb, rH, rF, hdiag1, ppa, ppb, h1, f1, nGe, nGsGe);
+        if constexpr (SW_DUAL && (Q2 || PW || (SW_DUAL_LONG && LINKED))) {  // measured: +3% for the query-pair mode, -2% with the PRMT (mode 0)
+          gotoh_rows_dual<R, Q2, US, PW>(HA, E, best, hdiag, pa, pb, rH, rF, hdiag1, ppa, ppb, h1, f1, nGe, nGsGe,
+                                         wmul);
         } else {
           // sub-lane 1 (rows RH..R-1, column t-1) first: it reads rows it owns only
           gotoh_rows_inplace<R, RH, R, Q2, US>(HA, E, best, hdiag1, ppa, ppb, h1, f1, nGe, nGsGe);
@@ -380,12 +383,11 @@ __device__ __forceinline__ void emit_pair(const InterArgs& a, const QueryDesc& d
 //   then (query, CHUNK of NT/G short pairs) -- one pair per lane group
 //     (inter-task mode).
 // Queries are in descending length, pairs in descending length.
-template <int G, int R, int NT>
-#ifdef SW_MINB  // experiments only: __launch_bounds__(NT, 1) lets ptxas take 225 registers (1 CTA/SM, -5% on config 3)
-__global__ void __launch_bounds__(NT, SW_MINB) inter_kernel(InterArgs a) {
-#else
-__global__ void __launch_bounds__(NT) inter_kernel(InterArgs a) {
-#endif
+// PWK = 1: the variant whose single-query slots use the wide profile (a separate
+// instantiation: its pair build needs more live registers, which must not raise
+// the register allocation of the default kernel).
+template <int G, int R, int NT, int PWK>
+__device__ __forceinline__ void inter_body(InterArgs a) {
   extern __shared__ __align__(16) uint8_t smem[];
   // An item is either short or long, so the two uses share shared memory:
   uint8_t* sprof = smem;                         // short mode: the strip profile (bank-spread copies)
@@ -561,6 +563,7 @@ __global__ void __launch_bounds__(NT) inter_kernel(InterArgs a) {
       const SlotDesc d = a.slots[sl];
       const int chunk = sc.y;
       const bool q2 = d.mode == 1;
+      constexpr bool wide = PWK != 0 && R % 8 == 0;  // mode 0 with the 32-bit (query-pair layout) profile
       int p, half = 0;
       if (q2) {  // chunk of NG half-pairs: DB sequence = one half of a pair
         const int hp = chunk * NG + g;
@@ -577,9 +580,10 @@ __global__ void __launch_bounds__(NT) inter_kernel(InterArgs a) {
       int T = pr.len + G * SubLanes<R>::V;         // the last sub-lane finishes column len-1 at step T-2
       if (G < 32) T = __reduce_max_sync(FULL, T);  // warp-uniform trip count (shuffles)
       uint32_t best = 0;
-      const int SBx = q2 ? a.SB2 : a.SB;
-      const int ncp = q2 ? a.ncopy[1] : a.ncopy[0], csx = q2 ? a.cstride[1] : a.cstride[0];
-      const uint32_t skw = q2 ? 0u : a.cskew0;
+      const bool l2 = q2 || wide;  // query-pair profile geometry
+      const int SBx = l2 ? a.SB2 : a.SB;
+      const int ncp = l2 ? a.ncopy[1] : a.ncopy[0], csx = l2 ? a.cstride[1] : a.cstride[0];
+      const uint32_t skw = l2 ? 0u : a.cskew0;
       const int rs = d.res_stride;  // > 0: every strip of the slot resident (loaded once per slot)
       for (int s = 0; s < d.n_strips; ++s) {
         const int want = rs ? ((sl << 16) | 0xffff) : ((sl << 16) | s);
@@ -635,8 +639,13 @@ __global__ void __launch_bounds__(NT) inter_kernel(InterArgs a) {
             best &= (si.emit0 >= 0 ? 0xffff0000u : 0xffffffffu) & (si.emit1 >= 0 ? 0x0000ffffu : 0xffffffffu);
           }
         } else {
-          strip_pass<G, R, false>(gprof, a.LS, a.LB, a.stream + pr.off, pr.len, T, k, s > 0, s + 1 < d.n_strips,
-                                  bb, bb, Link{}, a.code_pad2, a.nGe, a.nGsGe, best);
+          if constexpr (wide)
+            strip_pass<G, R, false, false, 16, 1>(gprof, a.LS2, a.LB2, a.stream + pr.off, pr.len, T, k, s > 0,
+                                                  s + 1 < d.n_strips, bb, bb, Link{}, a.code_pad2, a.nGe, a.nGsGe,
+                                                  best, 0u, a.wmul);
+          else
+            strip_pass<G, R, false>(gprof, a.LS, a.LB, a.stream + pr.off, pr.len, T, k, s > 0, s + 1 < d.n_strips,
+                                    bb, bb, Link{}, a.code_pad2, a.nGe, a.nGsGe, best);
         }
       }
       if (!q2) {  // mode 0: one query, both halves are DB sequences
@@ -654,6 +663,20 @@ __global__ void __launch_bounds__(NT) inter_kernel(InterArgs a) {
   }
 }
 
+template <int G, int R, int NT>
+#ifdef SW_MINB  // experiments only: __launch_bounds__(NT, 1) lets ptxas take 225 registers (1 CTA/SM, -5% on config 3)
+__global__ void __launch_bounds__(NT, SW_MINB) inter_kernel(InterArgs a) {
+#else
+__global__ void __launch_bounds__(NT) inter_kernel(InterArgs a) {
+#endif
+  inter_body<G, R, NT, 0>(a);
+}
+// the wide-profile variant, held to 2 CTAs/SM (128 registers) like the default
+template <int G, int R, int NT>
+__global__ void __launch_bounds__(NT, 2) inter_kernel_wide(InterArgs a) {
+  inter_body<G, R, NT, 1>(a);
+}
+
 // ---------------------------------------------------------------------------
 // Instantiation table.
 #ifndef SW_INTER_NT
@@ -669,8 +692,17 @@ constexpr int INTER_NT = SW_INTER_NT;  // threads per CTA of the scoring kernel
 
 typedef void (*inter_fn)(InterArgs);
 
-static inter_fn pick_inter(int G, int R, int NT) {
+#define SW_WIDE_CASES(X) X(4, 24) X(8, 24) X(8, 16) X(16, 24) X(8, 32) X(4, 16)
+
+static inter_fn pick_inter(int G, int R, int NT, int wide = 0) {
   if (NT != INTER_NT) return nullptr;
+  if (wide) {
+#define X(g, r) \
+    if (G == g && R == r) return inter_kernel_wide<g, r, INTER_NT>;
+    SW_WIDE_CASES(X)
+#undef X
+    return nullptr;
+  }
 #define X(g, r) \
   if (G == g && R == r) return inter_kernel<g, r, INTER_NT>;
   SW_INTER_CASES(X)
@@ -679,10 +711,11 @@ static inter_fn pick_inter(int G, int R, int NT) {
 }
 
 bool inter_config_supported(int G, int R) { return pick_inter(G, R, INTER_NT) != nullptr; }
+bool inter_wide_supported(int G, int R) { return pick_inter(G, R, INTER_NT, 1) != nullptr; }
 int inter_block_threads() { return INTER_NT; }
 
-int inter_max_ctas_per_sm(int G, int R, int NT, int smem_bytes) {
-  inter_fn f = pick_inter(G, R, NT);
+int inter_max_ctas_per_sm(int G, int R, int NT, int smem_bytes, int wide) {
+  inter_fn f = pick_inter(G, R, NT, wide);
   if (!f) return 0;
   if (smem_bytes > 48 * 1024)
     cudaFuncSetAttribute(f, cudaFuncAttributeMaxDynamicSharedMemorySize, smem_bytes);
@@ -691,8 +724,9 @@ int inter_max_ctas_per_sm(int G, int R, int NT, int smem_bytes) {
   return n;
 }
 
-cudaError_t launch_inter(int G, int R, int NT, int grid, int smem_bytes, const InterArgs& a, cudaStream_t st) {
-  inter_fn f = pick_inter(G, R, NT);
+cudaError_t launch_inter(int G, int R, int NT, int grid, int smem_bytes, const InterArgs& a, cudaStream_t st,
+                         int wide) {
+  inter_fn f = pick_inter(G, R, NT, wide);
   if (!f) return cudaErrorInvalidValue;
   if (smem_bytes > 48 * 1024) {
     cudaError_t e = cudaFuncSetAttribute(f, cudaFuncAttributeMaxDynamicSharedMemorySize, smem_bytes);

@@ -149,14 +149,28 @@ __device__ __forceinline__ void gotoh_rows_inplace(uint32_t (&H)[R], uint32_t (&
 }
 
 // Profile values S(q_r, letter) of rows [R0, R1) for one lane (see gotoh_rows_inplace).
-template <int R, int R0, int R1, bool Q2, int US>
-__device__ __forceinline__ void load_rows(uint32_t (&sv)[R1 - R0], uint32_t pa, uint32_t pb) {
+// PW (wide single-query profile): 32-bit rows holding S & 0xffff; the pair
+// (S[b] : S[a]) is one IMAD, S[b] * 2^16 + S[a], on the FMA pipe instead of a
+// PRMT on the ALU pipe (wmul = 65536, a runtime value so that it stays an IMAD).
+__device__ __forceinline__ uint32_t imad_u32(uint32_t a, uint32_t b, uint32_t c) {
+  uint32_t d;
+  asm("mad.lo.u32 %0, %1, %2, %3;" : "=r"(d) : "r"(a), "r"(b), "r"(c));
+  return d;
+}
+
+template <int R, int R0, int R1, bool Q2, int US, int PW = 0>
+__device__ __forceinline__ void load_rows(uint32_t (&sv)[R1 - R0], uint32_t pa, uint32_t pb, uint32_t wmul = 0) {
   constexpr int N = R1 - R0;
-  constexpr int UB = Q2 ? 4 : ((R % 8 == 0 && R0 % 8 == 0 && N % 8 == 0) ? 8 : 4);
+  constexpr int UB = (Q2 || PW) ? 4 : ((R % 8 == 0 && R0 % 8 == 0 && N % 8 == 0) ? 8 : 4);
 #pragma unroll
   for (int u = R0 / UB; u < R1 / UB; ++u) {
     const int b = u * UB - R0;
-    if constexpr (Q2) {
+    if constexpr (PW) {
+      const uint4 x = lds128(pa + u * US);
+      const uint4 y = lds128(pb + u * US);
+      sv[b] = imad_u32(y.x, wmul, x.x); sv[b + 1] = imad_u32(y.y, wmul, x.y);
+      sv[b + 2] = imad_u32(y.z, wmul, x.z); sv[b + 3] = imad_u32(y.w, wmul, x.w);
+    } else if constexpr (Q2) {
       const uint4 w = lds128(pa + u * US);
       sv[b] = w.x; sv[b + 1] = w.y; sv[b + 2] = w.z; sv[b + 3] = w.w;
     } else if constexpr (UB == 8) {
@@ -180,16 +194,17 @@ __device__ __forceinline__ void load_rows(uint32_t (&sv)[R1 - R0], uint32_t pa, 
 // Hio1 / Fio1 are sub-lane 0's outputs of the previous step).  The two F
 // chains are independent, so emitting their rows alternately hands the
 // scheduler two ready instructions per dependency step.
-template <int R, bool Q2, int US>
+template <int R, bool Q2, int US, int PW = 0>
 __device__ __forceinline__ void gotoh_rows_dual(uint32_t (&H)[R], uint32_t (&E)[R], uint32_t& best,
                                                 uint32_t& hdiag0, uint32_t pa0, uint32_t pb0, uint32_t& Hio0,
                                                 uint32_t& Fio0, uint32_t& hdiag1, uint32_t pa1, uint32_t pb1,
-                                                uint32_t& Hio1, uint32_t& Fio1, uint32_t nGe, uint32_t nGsGe) {
+                                                uint32_t& Hio1, uint32_t& Fio1, uint32_t nGe, uint32_t nGsGe,
+                                                uint32_t wmul = 0) {
   constexpr int RH = R / 2;
   static_assert(R % 8 == 0, "two sub-lanes of whole 4-row units");
   uint32_t s0[RH], s1[RH];
-  load_rows<R, 0, RH, Q2, US>(s0, pa0, pb0);
-  load_rows<R, RH, R, Q2, US>(s1, pa1, pb1);
+  load_rows<R, 0, RH, Q2, US, PW>(s0, pa0, pb0, wmul);
+  load_rows<R, RH, R, Q2, US, PW>(s1, pa1, pb1, wmul);
   uint32_t F0 = Fio0, F1 = Fio1;
   uint32_t d0 = __vadd2(hdiag0, s0[0]);
   uint32_t d1 = __vadd2(hdiag1, s1[0]);

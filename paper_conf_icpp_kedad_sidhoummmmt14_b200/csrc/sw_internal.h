@@ -108,6 +108,8 @@ struct SlotDesc {
   int n_items;               // short work items of this slot
   int pair_begin;            // short pairs of this slot: [pair_begin, pair_end)
   int res_stride;            // > 0: all strips resident in smem, strip s at s * res_stride (bytes)
+  int wide;                  // mode 0 with the 32-bit profile (S & 0xffff per row, query-pair geometry)
+  int pad_;
 };
 
 struct InterArgs {
@@ -127,6 +129,7 @@ struct InterArgs {
   // per-copy bank skew of the mode-0 copies: copy c sits at c * cstride[0] +
   // 4 * ((cskew0 >> 8c) & 0xff) (0 for the linear layout; mode 1 is always linear)
   uint32_t cskew0;
+  uint32_t wmul;             // 65536 (runtime, so the wide mode's pair build stays an IMAD)
   int SBL, LSL, LBL;         // long geometry (32 lanes x LONG_R rows)
   int n_long_items;          // sum over queries of n_long * n_super
   uint2* links;              // [gridDim][NT/32][lcap] strip-to-strip rows inside a CTA (long items)
@@ -180,8 +183,10 @@ cudaError_t launch_build_profile(const uint8_t* q, int m, const int8_t* matrix, 
 cudaError_t launch_build_profile_q2(const uint8_t* qa, int ma, const uint8_t* qb, int mb, const int8_t* matrix,
                                     int alpha, int G, int R, int LB2, int LS2, int n_strips, int SB2, uint8_t* prof,
                                     cudaStream_t st);
-int inter_max_ctas_per_sm(int G, int R, int NT, int smem_bytes);
-cudaError_t launch_inter(int G, int R, int NT, int grid, int smem_bytes, const InterArgs& a, cudaStream_t st);
+int inter_max_ctas_per_sm(int G, int R, int NT, int smem_bytes, int wide = 0);
+cudaError_t launch_inter(int G, int R, int NT, int grid, int smem_bytes, const InterArgs& a, cudaStream_t st,
+                         int wide = 0);
+bool inter_wide_supported(int G, int R);
 bool inter_config_supported(int G, int R);
 int inter_block_threads();  // NT of the scoring kernel (its long items use NT/32 chained warps)
 cudaError_t launch_rescore(int grid, const RescoreArgs& a, cudaStream_t st);

@@ -261,6 +261,19 @@ def test_query_packing(pack, thr):
     np.testing.assert_array_equal(got, oracle_scores(qc, qo, dc, do))
 
 
+@pytest.mark.parametrize("G,R", [(8, 24), (4, 24), (8, 16), (16, 24), (8, 32), (4, 16)])
+def test_wide_single_query_profile(G, R):
+    """Single-query mode with the wide profile (option wide_profile: 32-bit rows,
+    the (S[b] : S[a]) pair built by one IMAD instead of a PRMT; its own kernel
+    instantiation); multi-strip queries, ragged DB, PAD columns."""
+    rng = np.random.default_rng(81 + G + R)
+    dc, do = _seqs(list(rng.integers(1, 350, size=120)) + [0, 1, 3], rng, alpha=24)
+    qc, qo = _seqs([3 * G * R + 7, G * R, 17, 1], rng, alpha=24)
+    opts = {"wide_profile": 1, "query_pairs": 0, "force_G": G, "force_R": R}
+    got = gpu_scores(qc, qo, dc, do, opts=opts)
+    np.testing.assert_array_equal(got, oracle_scores(qc, qo, dc, do))
+
+
 @pytest.mark.parametrize("skew", [0, 1])
 @pytest.mark.parametrize("G,R", [(8, 24), (8, 8), (16, 24), (16, 8), (8, 12), (4, 16), (8, 16)])
 def test_single_query_profile_copies(G, R, skew):

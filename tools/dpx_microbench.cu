@@ -112,6 +112,43 @@ __global__ void k_cell2(uint32_t* out, uint32_t seed) {
   if (best == 0x12345678u) out[blockIdx.x] = best;
 }
 
+// k_cell2 with NCH independent F chains per thread (rows interleaved chain by
+// chain, as gotoh_rows_dual does for NCH = 2): how far more ILP per warp lifts
+// the latency-bound cell rate at a fixed occupancy.
+template <int R, int NCH>
+__global__ void k_cellN(uint32_t* out, uint32_t seed) {
+  constexpr int RC = R / NCH;
+  uint32_t H[R], E[R], S[R];
+  const uint32_t nge = 0xfffefffeu, ngsge = 0xfff4fff4u;
+#pragma unroll
+  for (int r = 0; r < R; ++r) { H[r] = (seed + r) & 0x00ff00ffu; E[r] = 0; S[r] = ((r * 3 + threadIdx.x) & 7) * 0x00010001u; }
+  uint32_t best = 0, hdiag = 0;
+  for (int it = 0; it < ITERS / 4; ++it) {
+    uint32_t F[NCH], hd[NCH], dprev[NCH];
+#pragma unroll
+    for (int c = 0; c < NCH; ++c) { F[c] = 0; hd[c] = hdiag + c; dprev[c] = 0; }
+#pragma unroll
+    for (int i = 0; i < RC; ++i) {
+#pragma unroll
+      for (int c = 0; c < NCH; ++c) {
+        const int r = c * RC + i;
+        const uint32_t dg = __vadd2(hd[c], S[r]);
+        const uint32_t h = __vimax3_s16x2(dg, E[r], F[c]);
+        const uint32_t t = __vadd2(h, ngsge);
+        E[r] = __viaddmax_s16x2_relu(E[r], nge, t);
+        F[c] = __viaddmax_s16x2_relu(F[c], nge, t);
+        hd[c] = H[r]; H[r] = h;
+        if (i & 1) best = __vimax3_s16x2(best, dprev[c], dg); else dprev[c] = dg;
+      }
+    }
+    uint32_t x = 0;
+#pragma unroll
+    for (int c = 0; c < NCH; ++c) x ^= F[c];
+    hdiag = x ^ it;
+  }
+  if (best == 0x12345678u) out[blockIdx.x] = best;
+}
+
 __global__ void k_clock(unsigned long long* t) {
   unsigned long long c0 = clock64();
   uint32_t x = threadIdx.x;
@@ -182,6 +219,17 @@ int main() {
     float mc = time_kernel(k_cell2<24, false>, sms * g, block, d_out);
     double cells = double(sms * g) * block * (ITERS / 4) * 24 * 2;
     printf("{\"probe\":\"gotoh_cellpair_D_max3_R24\",\"blocks_per_sm\":%d,\"ms\":%.4f,\"GCUPS\":%.1f}\n", g, mc, cells / (mc * 1e6));
+  }
+  for (int g = 1; g <= 4; g *= 2) {
+    const double cells = double(sms * g) * block * (ITERS / 4) * 24 * 2;
+    float mc = time_kernel(k_cellN<24, 1>, sms * g, block, d_out);
+    printf("{\"probe\":\"gotoh_cellpair_R24_chains1\",\"blocks_per_sm\":%d,\"ms\":%.4f,\"GCUPS\":%.1f}\n", g, mc, cells / (mc * 1e6));
+    mc = time_kernel(k_cellN<24, 2>, sms * g, block, d_out);
+    printf("{\"probe\":\"gotoh_cellpair_R24_chains2\",\"blocks_per_sm\":%d,\"ms\":%.4f,\"GCUPS\":%.1f}\n", g, mc, cells / (mc * 1e6));
+    mc = time_kernel(k_cellN<24, 3>, sms * g, block, d_out);
+    printf("{\"probe\":\"gotoh_cellpair_R24_chains3\",\"blocks_per_sm\":%d,\"ms\":%.4f,\"GCUPS\":%.1f}\n", g, mc, cells / (mc * 1e6));
+    mc = time_kernel(k_cellN<24, 4>, sms * g, block, d_out);
+    printf("{\"probe\":\"gotoh_cellpair_R24_chains4\",\"blocks_per_sm\":%d,\"ms\":%.4f,\"GCUPS\":%.1f}\n", g, mc, cells / (mc * 1e6));
   }
   CK(cudaGetLastError());
   return 0;

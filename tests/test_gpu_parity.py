@@ -204,6 +204,19 @@ def test_intra_task_mode_forced():
     np.testing.assert_array_equal(got, oracle_scores(qc, qo, dc, do))
 
 
+def test_intra_task_packed_long_pairs():
+    """Option pack_long: a query with fewer intra-task strips than warps scores
+    W / S long pairs per CTA item (S warps per pair); odd pair counts leave a
+    partly filled last item."""
+    rng = np.random.default_rng(23)
+    dl = list(rng.integers(1, 900, size=75)) + [0, 1, 65, 66, 67]
+    dc, do = _seqs(dl, rng)
+    ql = [1, 100, 511, 512, 513, 1500, 2100, 4100]   # 1, 1, 1, 1, 2, 3, 5, 9 strips of 512 rows
+    qc, qo = _seqs(ql, rng)
+    got = gpu_scores(qc, qo, dc, do, opts={"t_long": 64, "pack_long": 1})
+    np.testing.assert_array_equal(got, oracle_scores(qc, qo, dc, do))
+
+
 def test_long_db_sequences():
     rng = np.random.default_rng(22)
     dl = list(rng.integers(3001, 6000, size=24)) + list(rng.integers(1, 400, size=60))

@@ -206,6 +206,10 @@ int32_t sw_last_stats(sw_handle_t h, sw_stats_t* out);
  *                         pair > 3000 when such pairs hold most of the residues)
  *   "pack_long"           1: pack several long pairs per CTA when a query has
  *                         fewer intra-task strips than warps (default 0)
+ *   "bank_copy"           1: shared-memory strip profiles as bank-spread copies
+ *                         with 128-byte letter rows (default 1), 0: one copy
+ *   "pack_queries"        1: a query-pair slot's shorter half carries further
+ *                         queries laid end to end on strip boundaries (default 1)
  *   "bank_skew"           1: single-query profile copies one per lane group of
  *                         a shared-memory phase at searched bank skews
  *                         (conflict-free; default 1), 0: the linear layout

@@ -217,6 +217,19 @@ def test_intra_task_packed_long_pairs():
     np.testing.assert_array_equal(got, oracle_scores(qc, qo, dc, do))
 
 
+@pytest.mark.parametrize("pairs", [0, 1])
+@pytest.mark.parametrize("G,R", [(4, 24), (8, 24), (16, 12)])
+def test_profile_without_bank_copies(G, R, pairs):
+    """Option bank_copy 0: one shared-memory copy of the strip profile, unpadded
+    letter rows (the layout the bank-spread copies replace)."""
+    rng = np.random.default_rng(91 + G + R + pairs)
+    dc, do = _seqs(list(rng.integers(1, 400, size=100)) + [0, 2], rng)
+    qc, qo = _seqs([2 * G * R + 5, 40, G * R], rng)
+    opts = {"bank_copy": 0, "query_pairs": pairs, "force_G": G, "force_R": R}
+    got = gpu_scores(qc, qo, dc, do, opts=opts)
+    np.testing.assert_array_equal(got, oracle_scores(qc, qo, dc, do))
+
+
 def test_long_db_sequences():
     rng = np.random.default_rng(22)
     dl = list(rng.integers(3001, 6000, size=24)) + list(rng.integers(1, 400, size=60))

@@ -177,3 +177,49 @@ def random_seqs(rng: np.random.Generator, n: int, lmin: int, lmax: int, alpha: i
     np.cumsum(lens, out=off[1:])
     codes = rng.integers(0, alpha, size=int(off[-1])).astype(np.uint8)
     return codes, off
+
+
+def subset(codes, off, ids):
+    """Sequences `ids` (in that order) of a (codes, offsets) set: (codes, offsets)."""
+    ids = np.asarray(ids, dtype=np.int64)
+    lens = off[ids + 1] - off[ids]
+    so = np.zeros(len(ids) + 1, dtype=np.int64)
+    np.cumsum(lens, out=so[1:])
+    sc = np.empty(int(so[-1]), dtype=np.uint8)
+    for k, i in enumerate(ids):
+        sc[so[k]:so[k + 1]] = codes[off[i]:off[i + 1]]
+    return sc, so
+
+
+def c5_sample(doff, n_queries: int, per_stratum: int = 625, seed: int = 0xC5):
+    """SURVEY.md 8(d) C5 sampling plan (input selection only, no SW arithmetic).
+
+    Strata = query x DB-length decile x DB-index octile (the 8 contiguous index
+    ranges stand for the 8 shards of the input order): 20 x 10 x 8 = 1,600
+    strata of `per_stratum` distinct sequences each (10^6 pairs at the defaults).
+    Returns dict(q, d, stratum) int64 arrays sorted by (stratum, d), and cells.
+    """
+    doff = np.asarray(doff, dtype=np.int64)
+    nd = len(doff) - 1
+    lens = np.diff(doff)
+    edges = np.quantile(lens, np.linspace(0, 1, 11)[1:-1], method="lower")
+    dec = np.searchsorted(edges, lens, side="right")               # 0..9
+    octl = (np.arange(nd, dtype=np.int64) * 8) // max(nd, 1)        # 0..7
+    key = dec * 8 + octl
+    order = np.argsort(key, kind="stable")
+    bounds = np.searchsorted(key[order], np.arange(81))
+    qs, ds, ss = [], [], []
+    for qi in range(n_queries):
+        for k in range(80):
+            pool = order[bounds[k]:bounds[k + 1]]
+            if not len(pool):
+                continue
+            rng = np.random.default_rng([seed, qi, k])
+            pick = np.sort(rng.choice(pool, size=min(per_stratum, len(pool)), replace=False))
+            qs.append(np.full(len(pick), qi, dtype=np.int64))
+            ds.append(pick.astype(np.int64))
+            ss.append(np.full(len(pick), qi * 80 + k, dtype=np.int64))
+    q = np.concatenate(qs) if qs else np.zeros(0, np.int64)
+    d = np.concatenate(ds) if ds else np.zeros(0, np.int64)
+    s = np.concatenate(ss) if ss else np.zeros(0, np.int64)
+    return dict(q=q, d=d, stratum=s, cells=0.0)

@@ -134,3 +134,53 @@ def score_cigar(q, d, q_begin: int, d_begin: int, ops, S, gs: int, ge: int) -> i
         else:
             s -= gs + k * ge; j += k
     return s
+
+
+def rule_alignment(q, d, S, gs: int, ge: int):
+    """The best local alignment that reading R-13 selects, from the exhaustive
+    enumeration (no DP matrices): among all optimal alignments, the end cell
+    with the smallest j, then the smallest i; then, reading the alignment
+    BACKWARDS from its end, the lexicographically smallest token sequence where
+    at an aligned position the next token ranks STOP < M (diagonal) < D (gap in
+    the query, E) < I (gap in the subject, F), and inside a gap run CLOSE (the
+    run opens here) < EXTEND.  For Gs > 0 an optimal alignment has at most one
+    I run and one D run between consecutive aligned pairs, so expanding every
+    optimal chain of aligned pairs into its (one or two) gap orders lists them
+    all.  Returns (score, q_begin, q_end, d_begin, d_end, ops) like
+    oracle.gotoh_align, ops run-length (len << 2 | op), op 0 = M, 1 = I, 2 = D."""
+    assert gs > 0, "the expansion below assumes Gs > 0"
+    best, chains = brute_local_chains(q, d, S, gs, ge)
+    if best == 0:
+        return (0, -1, -1, -1, -1, [])
+    end = min((c[-1][1], c[-1][0]) for c in chains)
+    STOP, M, D, I = 0, 1, 2, 3
+    CLOSE, EXT = 0, 1
+    cands = []
+    for c in chains:
+        if (c[-1][1], c[-1][0]) != end:
+            continue
+        variants = [([], [])]           # (backward tokens, backward ops)
+        for k in range(len(c) - 1, -1, -1):
+            variants = [(t + [M], o + ["M"]) for t, o in variants]
+            if k == 0:
+                variants = [(t + [STOP], o) for t, o in variants]
+                break
+            di = c[k][0] - c[k - 1][0] - 1
+            dj = c[k][1] - c[k - 1][1] - 1
+            runD = ([D] + [EXT] * (dj - 1) + [CLOSE], ["D"] * dj) if dj else ([], [])
+            runI = ([I] + [EXT] * (di - 1) + [CLOSE], ["I"] * di) if di else ([], [])
+            orders = [(runD, runI), (runI, runD)] if (di and dj) else [(runD, runI)]
+            variants = [(t + a[0] + b[0], o + a[1] + b[1]) for t, o in variants for a, b in orders]
+        cands += [(t, o, c) for t, o in variants]
+    tok, bops, c = min(cands, key=lambda x: x[0])
+    fwd = bops[::-1]
+    ops, run, prev = [], 0, None
+    code = {"M": 0, "I": 1, "D": 2}
+    for op in fwd + [None]:
+        if op == prev:
+            run += 1
+            continue
+        if prev is not None:
+            ops.append((run << 2) | code[prev])
+        prev, run = op, 1
+    return (best, c[0][0], c[-1][0], c[0][1], c[-1][1], ops)

@@ -254,3 +254,75 @@ def test_align_fig1_linear_gaps():
     sc, qb, qe, db, de, ops = oracle.gotoh_align(q, d, S, 0, 2)
     assert sc == 5
     assert brute.score_cigar(q, d, qb, db, ops, S, 0, 2) == 5
+
+
+def test_align_tie_breaks_vs_enumeration():
+    """The WHOLE returned alignment -- end cell, start cell and every op, i.e.
+    the traceback's tie-breaks of reading R-13 (diagonal > E > F at an aligned
+    position, opening > extending inside a gap, stop at the first zero prefix) --
+    equals the one brute.rule_alignment selects by lexicographic order over the
+    exhaustively enumerated optimal alignments (no DP).  Small alphabets and
+    matrices with many equal entries make ties frequent."""
+    rng = np.random.default_rng(507)
+    n_ties = 0
+    for _ in range(400):
+        alpha = int(rng.integers(2, 4))
+        m, n = int(rng.integers(1, 7)), int(rng.integers(1, 7))
+        q = rng.integers(0, alpha, size=m).astype(np.uint8)
+        d = rng.integers(0, alpha, size=n).astype(np.uint8)
+        S = rng.choice([-2, -1, 0, 1, 2, 3], size=(alpha, alpha)).astype(np.int32)
+        gs, ge = int(rng.integers(1, 4)), int(rng.integers(0, 3))
+        got = oracle.gotoh_align(q, d, S, gs, ge)
+        exp = brute.rule_alignment(q, d, S, gs, ge)
+        assert got == exp, (q.tolist(), d.tolist(), S.tolist(), gs, ge, got, exp)
+        best, chains = brute.brute_local_chains(q, d, S, gs, ge)
+        n_ties += len(chains) > 1
+    assert n_ties > 100   # the sample really exercises the tie-breaks
+
+
+def _abcxy_matrix():
+    """a b c x y: a/a = c/c = 10, a/b = b/a = 9, every other pair -10."""
+    S = np.full((5, 5), -10, dtype=np.int32)
+    S[0, 0] = S[2, 2] = 10
+    S[0, 1] = S[1, 0] = 9
+    return S
+
+
+@pytest.mark.parametrize("case", [
+    # (query, subject, Gs, Ge, expected (score, qb, qe, db, de), expected ops); derivations in the docstring
+    ("ac", "abc", 1, 0, (19, 0, 1, 1, 2), ["2M"]),
+    ("axc", "ayc", 1, 1, (16, 0, 2, 0, 2), ["1M", "1I", "1D", "1M"]),
+    ("ac", "aaxc", 1, 0, (19, 0, 1, 1, 3), ["1M", "1D", "1M"]),
+    ("aaxc", "ac", 1, 0, (19, 1, 3, 0, 1), ["1M", "1I", "1M"]),
+    ("a", "aa", 1, 1, (10, 0, 0, 0, 0), ["1M"]),
+    ("aa", "a", 1, 1, (10, 0, 0, 0, 0), ["1M"]),
+])
+def test_align_tie_breaks_hand_derived(case):
+    """Hand-derived cases, matrix _abcxy_matrix():
+    1. diagonal vs E at an aligned position.  q=ac, d=abc, Gs 1, Ge 0: a-b then c-c
+       = 9 + 10 = 19, and a-a, gap over b, c-c = 10 - 1 + 10 = 19; no ungapped c pairs
+       better.  End (q1, d2) is unique; back at H(q0, d1) both the diagonal (a-b) and E
+       (b against a gap) reach 9: the diagonal wins -> q0-d1, q1-d2: ops 2M, db = 1.
+    2. E vs F.  q=axc, d=ayc, Gs 1, Ge 1: a-a, x against a gap, y against a gap, c-c =
+       20 - 2 - 2 = 16 (aligning x-y gives 10).  At H(q1, d1) H = E = F = 6 and the
+       diagonal (x-y) does not reach it: E first, so backwards the D run (y) comes
+       before the I run (x): forward M I D M.
+    3. open vs extend inside an E run.  q=ac, d=aaxc, Gs 1, Ge 0: q0 against d1 then a
+       one-residue gap (x), or q0 against d0 then a two-residue gap (a, x): both 19.
+       At E(q0, d2) opening from H(q0, d1) = 10 ties extending E(q0, d1) = 9: open ->
+       q0-d1, D, q1-d3: ops M D M, db = 1.
+    4. the same inside an F run (query and subject swapped): ops M I M, qb = 1.
+    5. end-cell tie in j: q=a, d=aa: 10 at (q0, d0) and (q0, d1): smallest j, d0.
+    6. end-cell tie in i: q=aa, d=a: 10 at (q0, d0) and (q1, d0): smallest i, q0.
+    (Stopping at the first zero prefix is covered by the enumeration test above.)
+    """
+    q, d, gs, ge, five, ops = case
+    S = _abcxy_matrix()
+    enc = {"a": 0, "b": 1, "c": 2, "x": 3, "y": 4}
+    qa = np.array([enc[x] for x in q], np.uint8)
+    da = np.array([enc[x] for x in d], np.uint8)
+    code = {"M": 0, "I": 1, "D": 2}
+    exp_ops = [(int(o[:-1]) << 2) | code[o[-1]] for o in ops]
+    got = oracle.gotoh_align(qa, da, S, gs, ge)
+    assert got == five + (exp_ops,)
+    assert brute.rule_alignment(qa, da, S, gs, ge) == got

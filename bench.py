@@ -2,12 +2,14 @@
 """bench.py -- whole-box GCUPS of the SWDUAL hot path on B200 (BASELINE.json metric).
 
 One step = one pass of the whole hot path over the workload: every (query,
-shard) task scored by sw_search on its GPU (profile build, inter-task DPX
-kernels, int32 re-score) plus the single collective, the all-gather of the
-int32 score blocks (N > 1).  Workload (default): BASELINE config 3, the 20-query
+shard) task scored by sw_search on its GPU (profile build, inter- and
+intra-task DPX kernels, int32 re-score) plus, at N > 1, the single collective
+(the all-gather of the int32 score blocks) and rank 0's merge (sw_assemble)
+into scores[Q][N] in the caller's order -- dist.ShardedSearch.step().  Workload (default): BASELINE config 3, the 20-query
 sweep (144..5478 aa) against the Swiss-Prot-sized synthetic DB (570k seqs,
 205M residues) -- the configuration the metric "GCUPS at 1/2/4/8 B200" is
-quoted on; the DB is cut into N shards and placed by the dual approximation.
+quoted on; at N > 1 the DB is cut into 4N shards whose (query, shard) tasks are
+placed on the GPUs by the dual approximation.
 
   python bench.py [--gpus N] [--steps K] [--warmup W] [--impl ours|reference]
   torchrun --nproc-per-node N bench.py --gpus N ...
@@ -69,9 +71,7 @@ def parse():
     ap.add_argument("--force-geom", default=None, help="G,R of the inter-task kernel (experiments; default auto)")
     ap.add_argument("--verify", type=int, default=0, help="after timing, check N sampled DB sequences "
                     "of the assembled scores against the CPU oracle (rank 0)")
-    ap.add_argument("--gather", default="nccl", choices=["nccl", "fused"],
-                    help="N > 1: all-gather of score blocks (nccl) or fused: every rank's scoring epilogue writes "
-                         "into rank 0's score matrix mapped over NVLink (CUDA IPC), no collective on the data path")
+    ap.add_argument("--shards", type=int, default=None, help="DB shards (default: 1 at N = 1, 4 per GPU at N > 1)")
     ap.add_argument("--dist-backend", default="nccl", help="nccl (default); gloo only for functional checks "
                     "of the multi-rank path on a box with fewer GPUs than ranks")
     return ap.parse_args()
@@ -142,20 +142,32 @@ def workload(args):
     return c, q_lens, d_lens
 
 
-def config_obj(args, c, q_lens, d_lens, n):
+def config_obj(args, c, q_lens, d_lens, n, n_shards=1):
     return {"workload": WORKLOADS[args.workload], "name": args.workload,
             "n_queries": int(len(q_lens)), "query_residues": int(q_lens.sum()),
             "n_db_seqs": int(len(d_lens)), "db_residues": int(d_lens.sum()),
             "matrix": "BLOSUM62", "gap_open": 10, "gap_extend": 2,
-            "shards": n, "placement": "dual-approximation (query, shard) tasks",
-            **({"gather": "fused epilogue into rank 0's matrix over CUDA IPC / NVLink" if args.gather == "fused"
-                else "NCCL all-gather of score blocks"} if n > 1 else {}),
+            "shards": n_shards, "placement": "dual-approximation (query, shard) tasks, calibrated task times",
+            **({"gather": "NCCL all-gather of the score blocks, then sw_assemble on rank 0 (caller-order "
+                          "scores[Q][N]) inside the timed step"} if n > 1 else {}),
             "l2": "inputs larger than L2: 205 MB packed DB > 126 MB L2, streamed once per query per step"
             if args.workload in ("c2", "c3", "t5hom", "t5het") and args.n_db is None else "small workload"}
 
 
-def cpu_baseline(c, target_cells: float, seed: int = 2024) -> dict:
-    """The oracle as it stands, on a bounded random sample of the workload's DB, all host cores."""
+def cpu_model() -> str:
+    try:
+        for ln in open("/proc/cpuinfo"):
+            if ln.startswith("model name"):
+                return ln.split(":", 1)[1].strip()
+    except OSError:
+        pass
+    return "unknown"
+
+
+def cpu_baseline(c, target_cells: float, seed: int = 2024, single_cells: float = 1.0e10) -> dict:
+    """The oracle as it stands, on a bounded random sample of the workload's DB,
+    all host cores (one single-threaded oracle process per core); plus the
+    single-core rate of SURVEY 8(d): all of C1, then a fixed 1e10-cell C2 sample."""
     import oracle
     from oracle.blosum62 import blosum62 as ob62
     d_lens = np.diff(c["doff"])
@@ -165,28 +177,36 @@ def cpu_baseline(c, target_cells: float, seed: int = 2024) -> dict:
     want_res = max(1.0, target_cells / max(qsum, 1))
     k = int(min(n, max(1, want_res / max(d_lens.mean(), 1))))
     idx = np.sort(rng.choice(n, size=k, replace=False))
-    lens = d_lens[idx]
-    off = np.zeros(k + 1, dtype=np.int64)
-    np.cumsum(lens, out=off[1:])
-    sub = np.concatenate([c["dcodes"][c["doff"][i]:c["doff"][i + 1]] for i in idx]) if k else np.zeros(0, np.uint8)
+    sub, off = swgen.subset(c["dcodes"], c["doff"], idx)
     cores = os.cpu_count() or 1
     oracle.build()
     t0 = time.perf_counter()
     oracle.gotoh_search(c["qcodes"], c["qoff"], sub, off, ob62(), 10, 2, procs=cores)
     dt = time.perf_counter() - t0
-    cells = float(qsum) * float(lens.sum())
-    # single core: one oracle process on ~1/cores of the same sample
-    k1 = max(1, k // cores)
-    off1 = off[:k1 + 1]
+    cells = float(qsum) * float(off[-1])
+    # single core: C1 in full + the first sequences of a seeded C2 sample up to single_cells
+    c1 = swgen.make_config("c1")
     t1 = time.perf_counter()
-    oracle.gotoh_search(c["qcodes"], c["qoff"], sub[:int(off1[-1])], off1, ob62(), 10, 2, procs=1)
+    oracle.gotoh_search(c1["qcodes"], c1["qoff"], c1["dcodes"], c1["doff"], ob62(), 10, 2, procs=1)
     dt1 = time.perf_counter() - t1
-    cells1 = float(qsum) * float(off1[-1])
+    cells1 = float(np.diff(c1["qoff"]).sum()) * float(c1["doff"][-1])
+    c2 = c if c.get("name") == "c2" else swgen.make_config("c2")
+    m2 = float(np.diff(c2["qoff"]).sum())
+    l2 = np.diff(c2["doff"])
+    idx2 = np.random.default_rng(seed + 1).permutation(len(l2))
+    k2 = int(np.searchsorted(np.cumsum(l2[idx2]) * m2, single_cells)) + 1
+    sub2, off2 = swgen.subset(c2["dcodes"], c2["doff"], np.sort(idx2[:k2]))
+    t2 = time.perf_counter()
+    oracle.gotoh_search(c2["qcodes"], c2["qoff"], sub2, off2, ob62(), 10, 2, procs=1)
+    dt2 = time.perf_counter() - t2
+    cells2 = m2 * float(off2[-1])
     return {"value": round(cells / dt / 1e9, 4), "unit": "GCUPS", "cores": cores, "kind": "oracle",
-            "sample": f"{k} seeded-random DB sequences ({int(lens.sum())} residues) x all {len(c['qoff']) - 1} queries "
-                      f"= {cells:.3e} cells in {dt:.1f} s",
-            "single_core": {"value": round(cells1 / dt1 / 1e9, 4), "unit": "GCUPS",
-                            "sample": f"first {k1} sequences of the sample = {cells1:.3e} cells in {dt1:.1f} s"}}
+            "cpu_model": cpu_model(),
+            "sample": f"{k} seeded-random DB sequences ({int(off[-1])} residues) x all {len(c['qoff']) - 1} queries "
+                      f"= {cells:.3e} cells in {dt:.1f} s on {cores} single-threaded oracle processes",
+            "single_core": {"value": round((cells1 + cells2) / (dt1 + dt2) / 1e9, 4), "unit": "GCUPS",
+                            "sample": f"C1 in full ({cells1:.3e} cells, {dt1:.1f} s) + {k2} seeded-random C2 "
+                                      f"sequences ({cells2:.3e} cells, {dt2:.1f} s), one process"}}
 
 
 def run_reference(args):
@@ -235,9 +255,8 @@ def run_ours(args):
     rank = int(os.environ.get("RANK", "0"))
     world = int(os.environ.get("WORLD_SIZE", "1"))
     local = int(os.environ.get("LOCAL_RANK", "0"))
-    if world != args.gpus:
-        if world == 1 and args.gpus > 1:
-            raise SystemExit("--gpus N > 1 needs torchrun --nproc-per-node N")
+    if world != args.gpus and world == 1 and args.gpus > 1:
+        raise SystemExit("--gpus N > 1 needs torchrun --nproc-per-node N")
     if args.dist_backend == "gloo":
         local = local % torch.cuda.device_count()  # functional check: ranks may share a GPU
     torch.cuda.set_device(local)
@@ -246,6 +265,9 @@ def run_ours(args):
     if world > 1:
         import torch.distributed as tdist
         if args.dist_backend == "nccl":
+            # communicator init lines (nranks, NVLS/NVLink transport) on stderr for the record
+            os.environ.setdefault("NCCL_DEBUG", "INFO")
+            os.environ.setdefault("NCCL_DEBUG_SUBSYS", "INIT")
             tdist.init_process_group("nccl", device_id=dev)
         else:
             tdist.init_process_group("gloo")
@@ -258,11 +280,6 @@ def run_ours(args):
     c, q_lens, d_lens = workload(args)
     Q, N = len(q_lens), len(d_lens)
     total_cells = float(q_lens.sum()) * float(d_lens.sum())
-    shards = swdist.shard_cut(c["doff"], world)
-    shard_res = [int(d_lens[s].sum()) for s in shards]
-    plan = swdist.place(q_lens, shards, shard_res, world)
-    blocks = swdist.local_blocks(plan, rank)
-
     S = sw.blosum62()
     h = sw.Handle(local, timing=True)
     for kv in filter(None, os.environ.get("SWDUAL_OPTS", "").split(",")):
@@ -272,67 +289,13 @@ def run_ours(args):
         fg, fr = (int(x) for x in args.force_geom.split(","))
         h.set_option("force_G", fg)
         h.set_option("force_R", fr)
-    fused = args.gather == "fused" and world > 1
-    full_dev = None
-    if fused:  # rank 0 owns scores[Q][N]; the other ranks map it (CUDA IPC; peer access over NVLink)
-        from torch.multiprocessing.reductions import reduce_tensor
-        if rank == 0:
-            full_dev = torch.zeros((Q, N), dtype=torch.int32, device=dev)
-            obj = [reduce_tensor(full_dev)]
-        else:
-            obj = [None]
-        pg.broadcast_object_list(obj, src=0)
-        if rank != 0:
-            fn, fargs = obj[0]
-            full_dev = fn(*fargs)
-    dbs = {}
-    for s, _qs in blocks:
-        sc, so = swdist.subset(c["dcodes"], c["doff"], shards[s])
-        if fused:  # scores land in columns shards[s] of rank 0's rows of N
-            dbs[s] = h.load_db(sc, so, alphabet_size=24, out_index=shards[s], out_n=N)
-        else:
-            dbs[s] = h.load_db(sc, so, alphabet_size=24)
-    # per block: query subset (host), device output view into one flat buffer
-    sizes = [swdist.flat_size(plan, r) for r in range(world)]
-    cap = max(max(sizes), 1)
-    flat = torch.zeros(cap, dtype=torch.int32, device=dev)
-    gathered = torch.empty(world * cap, dtype=torch.int32, device=dev) if world > 1 else None
-    jobs = []
-    pos = 0
-    for s, qs in blocks:
-        if fused:  # one search per run of consecutive queries: rows a..b of the shared matrix
-            runs, a0 = [], 0
-            for i in range(1, len(qs) + 1):
-                if i == len(qs) or qs[i] != qs[i - 1] + 1:
-                    runs.append(qs[a0:i])
-                    a0 = i
-            for run in runs:
-                qc, qo = swdist.subset(c["qcodes"], c["qoff"], run)
-                jobs.append((s, run, qc, qo, full_dev[run[0]:run[-1] + 1]))
-            continue
-        qc, qo = swdist.subset(c["qcodes"], c["qoff"], qs)
-        n = len(shards[s])
-        view = flat[pos:pos + len(qs) * n].view(len(qs), n)
-        pos += len(qs) * n
-        jobs.append((s, qs, qc, qo, view))
+    # the multi-GPU path (and, at N = 1, the single search): dist.ShardedSearch
+    ss = swdist.ShardedSearch(h, c["dcodes"], c["doff"], c["qcodes"], c["qoff"], S, 10, 2, rank=rank, world=world,
+                              n_shards=args.shards, pg=pg, backend=args.dist_backend)
     stream = torch.cuda.current_stream(dev)
 
-    def gather():
-        if args.dist_backend == "nccl":
-            pg.all_gather_into_tensor(gathered, flat)
-        else:  # gloo: host staging (functional checks only)
-            g = torch.empty(world * cap, dtype=torch.int32)
-            pg.all_gather_into_tensor(g, flat.cpu())
-            gathered.copy_(g)
-
-    def step():
-        for s, qs, qc, qo, view in jobs:
-            h.search(qc, qo, dbs[s], S, 10, 2, out=view, stream=stream)
-        if world > 1 and not fused:
-            gather()
-
     for _ in range(args.warmup):
-        step()
+        ss.step(stream)
     torch.cuda.synchronize()
     h.set_option("timing_accumulate", 1)
     h.set_option("timing_reset", 1)
@@ -344,7 +307,7 @@ def run_ours(args):
     e1 = torch.cuda.Event(enable_timing=True)
     e0.record(stream)
     for _ in range(args.steps):
-        step()
+        ss.step(stream)
     e1.record(stream)
     torch.cuda.synchronize()
     barrier()
@@ -352,109 +315,94 @@ def run_ours(args):
     ms_local = e0.elapsed_time(e1)
     st = h.last_stats()
     cdev = dev if args.dist_backend == "nccl" else torch.device("cpu")
-    ms = torch.tensor([ms_local], dtype=torch.float64, device=cdev)
-    if pg is not None:
-        pg.all_reduce(ms, op=pg.ReduceOp.MAX)
-    T = float(ms.item())
+
+    def allreduce(vals, op="sum"):
+        t = torch.tensor(vals, dtype=torch.float64, device=cdev)
+        if pg is not None:
+            pg.all_reduce(t, op=pg.ReduceOp.MAX if op == "max" else pg.ReduceOp.SUM)
+        return [float(x) for x in t.cpu()]
+
+    T = allreduce([ms_local], "max")[0]
     value = total_cells * args.steps / (T / 1e3) / 1e9
 
-    # dominant kernel: inter-task kernel over the short pairs (>= 95% of cells); the
-    # library's own accounting of one step gives its cells and the launch count
+    # dominant kernel: the persistent scoring launch of each search; the library's
+    # accounting of one step gives its cells and launches (rank-local, then summed)
     h.set_option("timing_accumulate", 0)
-    cells_step = 0.0
-    n_launch_step = 0
-    for s, qs, qc, qo, view in jobs:
-        h.search(qc, qo, dbs[s], S, 10, 2, out=view, stream=stream)
+    cells_local = 0.0
+    n_launch_local = 0
+    for s_, _qs, qc, qo, view in ss.jobs:
+        h.search(qc, qo, ss.dbs[s_], S, 10, 2, out=view, stream=stream)
         one = h.last_stats()
-        cells_step += one["cells"]
-        n_launch_step += one["n_launches"]
+        cells_local += one["cells"]
+        n_launch_local += one["n_launches"]
+    n_launch_local += 1 if ss.asm is not None else 0
     torch.cuda.synchronize()
-    if pg is not None:  # launches of every rank (the whole job)
-        nl = torch.tensor([n_launch_step], dtype=torch.int64, device=cdev)
-        pg.all_reduce(nl)
-        n_launch_step = int(nl.item())
+    cells_sum, kms_sum, nl_sum = allreduce([cells_local * args.steps, st["short_ms"], float(n_launch_local)])
     sm_max = clk.get("sm_max_mhz") or 1965.0
     n_sm = torch.cuda.get_device_properties(dev).multi_processor_count
     peak = n_sm * ALU_LANES_PER_SM_CLK * sm_max * 1e6 / OPS_PER_CELL / 1e9
-    achieved = cells_step * args.steps / (st["short_ms"] / 1e3) / 1e9 if st["short_ms"] > 0 else None
-    # algorithmic bytes of one launch: every query (pair) pass streams the packed DB once
-    # (~1 B per residue) and the int32 score matrix is written once
-    n_pass = (Q + 1) // 2 if Q > 1 else 1
-    alg_bytes = int(n_pass * int(d_lens.sum()) + 4 * Q * N)
+    achieved = cells_sum / (kms_sum / 1e3) / 1e9 if kms_sum > 0 else None   # per GPU
+    # algorithmic bytes of one scoring launch: the DB streamed once
+    # per query (1 B per residue per query) + the int32 scores written once
+    alg_bytes = int(Q * int(d_lens.sum()) + 4 * Q * N) // max(world, 1)
     traffic = None
     tpath = os.path.join(ROOT, "profiles", "traffic.json")
-    if os.path.exists(tpath) and args.n_db is None:  # the captured traffic is for the full-size workload
+    if os.path.exists(tpath) and args.n_db is None and world == 1:
         try:
             t = json.load(open(tpath)).get(args.workload)
             traffic = t.get("traffic_bytes_per_launch") if t else None
         except Exception:
             traffic = None
 
-    # e2e through the public API with host buffers
+    # e2e through the public API with host buffers: host queries (H2D inside sw_search)
+    # and the step's result read back to pinned host memory (rank 0)
     e2e = None
     if args.e2e_steps > 0:
-        host_out = {}
-        for s, qs, qc, qo, view in jobs:
-            host_out[s] = torch.empty(tuple(view.shape), dtype=torch.int32, pin_memory=True).numpy()
-        final_host = (torch.empty(Q * N if fused else world * cap, dtype=torch.int32, pin_memory=True)
-                      if world > 1 else None)
-        h2d = sum(int(qc.nbytes + qo.nbytes + S.nbytes) for _s, _q, qc, qo, _v in jobs)
-        d2h = sum(int(v.numel() * 4) for *_x, v in jobs) if world == 1 else (Q * N * 4 if fused else world * cap * 4)
-        def e2e_step():
-            if world == 1:
-                for s, qs, qc, qo, view in jobs:
-                    h.search(qc, qo, dbs[s], S, 10, 2, out=host_out[s], stream=stream)  # H2D + D2H inside
-            elif fused:
-                for s, qs, qc, qo, view in jobs:
-                    h.search(qc, qo, dbs[s], S, 10, 2, out=view, stream=stream)      # epilogue writes rank 0's rows
-                torch.cuda.synchronize()
-                barrier()
-                if rank == 0:
-                    final_host.copy_(full_dev.view(-1), non_blocking=False)
-            else:
-                for s, qs, qc, qo, view in jobs:
-                    h.search(qc, qo, dbs[s], S, 10, 2, out=view, stream=stream)      # H2D of queries inside
-                gather()
-                if rank == 0:
-                    final_host.copy_(gathered, non_blocking=False)
+        h2d = sum(int(qc.nbytes + qo.nbytes + S.nbytes) for _s, _q, qc, qo, _v in ss.jobs)
+        if world == 1 and len(ss.jobs) == 1:
+            host_out = [torch.empty(tuple(v.shape), dtype=torch.int32, pin_memory=True).numpy()
+                        for *_x, v in ss.jobs]
 
-        e2e_step()  # untimed: first host-output call allocates the library's staging buffer
+            def e2e_step():
+                ss.search_local(stream, host_out=host_out)      # sw_search with a host output: D2H inside
+            d2h = Q * N * 4
+        else:
+            final_host = torch.empty((Q, N), dtype=torch.int32, pin_memory=True) if rank == 0 else None
+
+            def e2e_step():
+                full = ss.step(stream)
+                if rank == 0:
+                    final_host.copy_(full, non_blocking=True)
+                torch.cuda.synchronize()
+            d2h = Q * N * 4
+        e2e_step()  # untimed: the first host-output call allocates the library's staging buffer
         barrier()
         torch.cuda.synchronize()
         t0 = time.perf_counter()
         for _ in range(args.e2e_steps):
             e2e_step()
         torch.cuda.synchronize()
-        dt = time.perf_counter() - t0
-        dtt = torch.tensor([dt], dtype=torch.float64, device=cdev)
-        if pg is not None:
-            pg.all_reduce(dtt, op=pg.ReduceOp.MAX)
-        e2e = {"value": round(total_cells * args.e2e_steps / float(dtt.item()) / 1e9, 2), "unit": "GCUPS",
-               "h2d_bytes_per_step": h2d * world, "d2h_bytes_per_step": d2h}
+        dt = allreduce([time.perf_counter() - t0], "max")[0]
+        e2e = {"value": round(total_cells * args.e2e_steps / dt / 1e9, 2), "unit": "GCUPS",
+               "h2d_bytes_per_step": int(allreduce([float(h2d)])[0]), "d2h_bytes_per_step": d2h,
+               "copies_declared": True}
 
     verified = None
     if args.verify > 0:
-        if world > 1 and not fused:
-            gather()
-            torch.cuda.synchronize()
-        if fused:
-            torch.cuda.synchronize()
-            barrier()
+        full = ss.step(stream)
+        torch.cuda.synchronize()
+        barrier()
         if rank == 0:
-            if fused:
-                full = full_dev.cpu().numpy()
-            else:
-                g = (gathered if world > 1 else flat).cpu().numpy().reshape(world, -1)
-                full = swdist.assemble(plan, Q, N, [g[r] for r in range(world)])
+            got = full.cpu().numpy()
             import oracle
             from oracle.blosum62 import blosum62 as ob62
             rng = np.random.default_rng(5)
             idx = np.sort(rng.choice(N, size=min(N, args.verify), replace=False))
-            sc, so = swdist.subset(c["dcodes"], c["doff"], idx)
+            sc, so = swgen.subset(c["dcodes"], c["doff"], idx)
             ref = oracle.gotoh_search(c["qcodes"], c["qoff"], sc, so, ob62(), 10, 2, procs=os.cpu_count() or 1)
-            verified = bool(np.array_equal(full[:, idx], ref))
+            verified = bool(np.array_equal(got[:, idx], ref))
             if not verified:
-                raise SystemExit(f"verify: {int((full[:, idx] != ref).sum())} mismatches vs oracle")
+                raise SystemExit(f"verify: {int((got[:, idx] != ref).sum())} mismatches vs oracle")
 
     cpu = None
     if rank == 0 and world == 1 and not args.no_cpu_baseline:
@@ -476,12 +424,13 @@ def run_ours(args):
         line = {"metric": METRIC, "value": round(value, 2), "unit": "GCUPS", "n_gpus": world, "steps": args.steps,
                 "warmup": args.warmup, "ms_per_step": round(T / args.steps, 3), "higher_is_better": True,
                 "scaling": "strong", "vs_baseline": None, "dtype": "int16x2 (DPX), int32 re-score",
-                "data": "synthetic", "config": config_obj(args, c, q_lens, d_lens, world),
+                "data": "synthetic", "config": config_obj(args, c, q_lens, d_lens, world, len(ss.shards)),
                 "roofline": {"bound": "alu", "achieved": round(achieved, 1) if achieved else None,
                              "peak": round(peak, 1), "unit": "GCUPS", "frac": round(achieved / peak, 4) if achieved else None,
                              "traffic": traffic,
                              "traffic_unit": "DRAM bytes per launch of the scoring kernel (profiles/traffic.json, ncu)",
                              "algorithmic_bytes_per_launch": alg_bytes,
+                             "algorithmic_bytes_basis": "SURVEY 8(d): 1 B per DB residue per query + 4 B per score",
                              "kernel": "inter_kernel (the persistent scoring launch: long and short pairs), CUDA events around each launch",
                              "peak_basis": f"{n_sm} SMs x {ALU_LANES_PER_SM_CLK} ALU-pipe lanes/clk x {sm_max:.0f} MHz / "
                                            f"{OPS_PER_CELL} ALU lane-ops per cell (minimal s16x2 Gotoh update; "
@@ -490,13 +439,12 @@ def run_ours(args):
                              "frac_vs_microbench": round(achieved / micro, 4) if (achieved and micro) else None,
                              "microbench_basis": "register-resident s16x2 cell update, same 3.5-ALU-op form, 2 CTAs/SM, "
                                                  "no memory or shuffles (profiles/r01_dpx_microbench.jsonl)"},
-                "cpu_baseline": cpu, "e2e": e2e, "gpu_launches": int(n_launch_step * args.steps),
+                "cpu_baseline": cpu, "e2e": e2e, "gpu_launches": int(nl_sum * args.steps),
                 **({"verified_sample": args.verify, "verified": verified} if args.verify else {}),
                 "clocks": clk,
                 "detail": {"search_ms_per_step": round(T / args.steps, 3),
-                           "short_kernel_ms_per_step": round(st["short_ms"] / args.steps, 3),
-                           "long_kernel_ms_per_step": round(st["long_ms"] / args.steps, 3),
-                           "cells_per_step": total_cells, "placement_makespan_model": plan.makespan}}
+                           "scoring_kernel_ms_per_step_per_gpu": round(kms_sum / max(world, 1) / args.steps, 3),
+                           "cells_per_step": total_cells, "placement_makespan_model_s": ss.plan.makespan}}
         print(json.dumps(line), flush=True)
     h.close()
     if pg is not None:

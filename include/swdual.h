@@ -77,8 +77,9 @@ int32_t sw_load_db(sw_handle_t h, const uint8_t* codes, const int64_t* offsets, 
  *   out_index   host, int64[n_seqs]: distinct output columns in [0, out_n).
  *   out_n       columns of the output rows (>= n_seqs).
  * sw_search on such a DB treats `scores` as int32[n_queries][out_n] (device or
- * peer-mapped memory only) and writes only this DB's columns, leaving the
- * others untouched.  sw_align keeps the caller's local DB indices.
+ * peer-mapped memory only) and writes only this DB's columns (every one of
+ * them, in every query row, including the zero rows of empty queries), leaving
+ * the others untouched.  sw_align keeps the caller's local DB indices.
  * Errors: as sw_load_db; SW_EINVAL for a bad mapping.
  */
 int32_t sw_load_db_mapped(sw_handle_t h, const uint8_t* codes, const int64_t* offsets, int64_t n_seqs,
@@ -95,8 +96,14 @@ int32_t sw_load_db_mapped(sw_handle_t h, const uint8_t* codes, const int64_t* of
  *   gap_open    Gs >= 0;  gap_extend  Ge >= 0;  Gs + Ge <= 32767.
  *   scores      host or device, int32[n_queries][n_seqs], row-major, in the
  *               caller's database order (the packer's length sort is undone).
- * Device `scores`: the call is stream-ordered on cuda_stream; the caller
- * synchronizes.  Host `scores`: the call returns after the results are copied.
+ * Device `scores`: the call is stream-ordered on cuda_stream and never blocks
+ * the host on the device (the int32 re-score kernel is always enqueued and reads
+ * the flagged-pair count on the device); the caller synchronizes.  Host
+ * `scores`: the call returns after the results are copied.
+ * Streams: the handle's scratch is shared by its searches; a search waits (on
+ * the device, cudaStreamWaitEvent) for the previous search of the same handle
+ * when that one ran on another stream, so concurrent calls on different streams
+ * are serialised on the device, never raced.  One host thread per handle.
  * Exactness: scores are exact int32; the int16 DPX path flags any pair whose
  * maximum reaches 32767 - max(matrix) and re-scores it in int32.
  * Errors: SW_EINVAL, SW_ESTATE (db from another handle), SW_ENOMEM, SW_ECUDA,
@@ -161,6 +168,33 @@ int32_t sw_align(sw_handle_t h, const uint8_t* q_codes, const int64_t* q_offsets
 int32_t sw_search_cpu(const uint8_t* q_codes, const int64_t* q_offsets, int32_t n_queries, const uint8_t* db_codes,
                       const int64_t* db_offsets, int64_t n_seqs, int32_t alphabet_size, const int8_t* matrix,
                       int32_t gap_open, int32_t gap_extend, int32_t n_threads, int32_t* scores);
+
+/*
+ * Merge of gathered score blocks into the full matrix (the
+ * master "merge[s]" the workers' results).  After the
+ * multi-GPU gather every rank's int32 blocks sit in one device buffer `src`;
+ * block b holds blocks[b].n_rows x blocks[b].n_cols scores (row-major) at
+ * src[src_off ..], its row i is query rows[row_off + i] and its column k is DB
+ * sequence cols[col_off + k] of the caller's order.  sw_assemble writes
+ * out[rows[..] * N + cols[..]] for every element, one kernel launch,
+ * stream-ordered; elements of `out` covered by no block are left untouched.
+ *   sw_assembly_create  host tables, copied to the device once (the layout is
+ *                       fixed for a placement); rows in [0, n_queries), cols in
+ *                       [0, N).  Free with sw_assembly_free (or sw_free).
+ *   sw_assemble         src: device int32[src_len] (>= every block's end);
+ *                       out: device int32[n_queries][N].
+ * Errors: SW_EINVAL (bad table, index out of range, src too short, NULL),
+ * SW_ENOMEM, SW_ECUDA.
+ */
+typedef struct sw_assembly_s* sw_assembly_t;
+typedef struct {
+  int64_t src_off, row_off, col_off, n_rows, n_cols;
+} sw_block_t;
+int32_t sw_assembly_create(sw_handle_t h, const sw_block_t* blocks, int32_t n_blocks, const int32_t* rows,
+                           int64_t n_rows, const int64_t* cols, int64_t n_cols, int32_t n_queries, int64_t N,
+                           sw_assembly_t* out);
+int32_t sw_assemble(sw_assembly_t a, const int32_t* src, int64_t src_len, int32_t* out, void* cuda_stream);
+int32_t sw_assembly_free(sw_assembly_t a);
 
 int32_t sw_free_db(sw_db_t db);
 int32_t sw_free(sw_handle_t h); /* frees the handle and any DBs still attached */
@@ -268,7 +302,8 @@ int32_t sw_schedule_dual(int64_t n_tasks, const double* p_cpu, const double* p_g
  * times rounded down to lambda / (4 n_tasks)); LPT on each side.  Makespan
  * <= (3/2 + 1/(4 n_gpu)) * lambda.  Same arguments and outputs as
  * sw_schedule_dual.  Time O(n^2 m k^2) per guess: SW_EUNSUPPORTED when the DP
- * would exceed ~4e9 state updates.
+ * table would exceed ~2.6e8 states (one byte each); SW_ENOMEM if the host
+ * allocation fails (no C++ exception crosses the ABI).
  */
 int32_t sw_schedule_dual_dp(int64_t n_tasks, const double* p_cpu, const double* p_gpu, int32_t n_cpu,
                             int32_t n_gpu, int32_t* out_pe, double* out_makespan, double* out_lambda);

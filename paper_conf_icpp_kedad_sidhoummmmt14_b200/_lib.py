@@ -16,7 +16,8 @@ SW_FLAG_TIMING = 1
 
 EXPORTS = ["sw_init", "sw_load_db", "sw_search", "sw_free_db", "sw_free", "sw_last_error",
            "sw_db_info", "sw_last_stats", "sw_set_option", "sw_encode_ascii", "sw_schedule_dual", "sw_align",
-           "sw_encode_nucleotide", "sw_search_cpu", "sw_schedule_dual_dp", "sw_load_db_mapped"]
+           "sw_encode_nucleotide", "sw_search_cpu", "sw_schedule_dual_dp", "sw_load_db_mapped",
+           "sw_assembly_create", "sw_assemble", "sw_assembly_free"]
 
 
 class SWError(RuntimeError):
@@ -29,6 +30,11 @@ class DbInfo(ctypes.Structure):
     _fields_ = [("n_seqs", ctypes.c_int64), ("n_residues", ctypes.c_int64), ("n_pairs", ctypes.c_int64),
                 ("n_long_pairs", ctypes.c_int64), ("max_len", ctypes.c_int64),
                 ("alphabet_size", ctypes.c_int32), ("device", ctypes.c_int32)]
+
+
+class Block(ctypes.Structure):
+    _fields_ = [("src_off", ctypes.c_int64), ("row_off", ctypes.c_int64), ("col_off", ctypes.c_int64),
+                ("n_rows", ctypes.c_int64), ("n_cols", ctypes.c_int64)]
 
 
 class Stats(ctypes.Structure):
@@ -83,6 +89,12 @@ def lib() -> ctypes.CDLL:
     L.sw_search_cpu.argtypes = [V, V, I32, V, V, I64, I32, V, I32, I32, I32, V]
     L.sw_align.restype = I32
     L.sw_align.argtypes = [V, V, V, I32, V, V, I32, V, I32, I32, V, V, V, V, V]
+    L.sw_assembly_create.restype = I32
+    L.sw_assembly_create.argtypes = [V, V, I32, V, I64, V, I64, I32, I64, P(V)]
+    L.sw_assemble.restype = I32
+    L.sw_assemble.argtypes = [V, V, I64, V, V]
+    L.sw_assembly_free.restype = I32
+    L.sw_assembly_free.argtypes = [V]
     _lib = L
     return L
 

@@ -13,7 +13,7 @@ import ctypes
 
 import numpy as np
 
-from ._lib import DbInfo, Stats, SW_FLAG_TIMING, check, lib
+from ._lib import Block, DbInfo, Stats, SW_FLAG_TIMING, check, lib
 
 try:  # torch is plumbing only (device buffers, streams)
     import torch
@@ -60,6 +60,28 @@ class Database:
             self.ptr = None
 
 
+class Assembly:
+    """sw_assembly_t: the fixed block layout of a multi-GPU placement."""
+
+    def __init__(self, handle: "Handle", ptr: ctypes.c_void_p):
+        self.handle = handle
+        self.ptr = ptr
+
+    def __call__(self, src, out, stream=None) -> None:
+        """sw_assemble: device src (gathered int32 blocks) -> device out [Q][N], stream-ordered."""
+        if not (torch is not None and isinstance(src, torch.Tensor) and isinstance(out, torch.Tensor)
+                and src.is_cuda and out.is_cuda and src.dtype == torch.int32 and out.dtype == torch.int32
+                and src.is_contiguous() and out.is_contiguous()):
+            raise ValueError("assemble: src and out must be contiguous int32 CUDA tensors")
+        check(lib().sw_assemble(self.ptr, ctypes.c_void_p(src.data_ptr()), src.numel(),
+                                ctypes.c_void_p(out.data_ptr()), _stream_ptr(stream)), self.handle.ptr)
+
+    def free(self) -> None:
+        if self.ptr:
+            lib().sw_assembly_free(self.ptr)
+            self.ptr = None
+
+
 class Handle:
     """sw_handle_t bound to one CUDA device."""
 
@@ -68,6 +90,7 @@ class Handle:
         check(lib().sw_init(int(device), SW_FLAG_TIMING if timing else 0, ctypes.byref(self.ptr)))
         self.device = int(device)
         self._dbs: list[Database] = []
+        self._asm: list["Assembly"] = []
 
     def set_option(self, key: str, value: int) -> None:
         check(lib().sw_set_option(self.ptr, key.encode(), int(value)), self.ptr)
@@ -90,6 +113,7 @@ class Handle:
                                           _stream_ptr(stream), ctypes.byref(out)), self.ptr)
         db = Database(self, out, n)
         db.out_n = n if out_index is None else int(out_n)
+        db.mapped = out_index is not None
         db.seq_lens = np.diff(offsets)
         self._dbs.append(db)
         return db
@@ -109,14 +133,25 @@ class Handle:
         N = getattr(db, "out_n", db.n_seqs)
         if out is None:
             if torch is not None and torch.cuda.is_available():
-                out = torch.empty((nq, N), dtype=torch.int32, device=f"cuda:{self.device}")
+                # a mapped DB writes only its own columns: the rest must not be garbage
+                alloc = torch.zeros if getattr(db, "mapped", False) else torch.empty
+                out = alloc((nq, N), dtype=torch.int32, device=f"cuda:{self.device}")
             else:
                 out = np.zeros((nq, N), dtype=np.int32)
         if torch is not None and isinstance(out, torch.Tensor):
-            assert out.dtype == torch.int32 and out.is_contiguous() and tuple(out.shape) == (nq, N)
-            optr = ctypes.c_void_p(out.data_ptr())
+            if out.dtype != torch.int32 or not out.is_contiguous() or tuple(out.shape) != (nq, N):
+                raise ValueError(f"search: out must be a contiguous int32 tensor of shape {(nq, N)}")
+            if out.is_cuda and out.device.index != self.device:
+                raise ValueError(f"search: out is on cuda:{out.device.index}, the handle on cuda:{self.device}")
+            if not out.is_cuda and not out.is_pinned():
+                out_np = out.numpy()                     # host tensor: written through its numpy view
+                optr = _vp(out_np)
+            else:
+                optr = ctypes.c_void_p(out.data_ptr())
         else:
-            assert out.dtype == np.int32 and out.flags.c_contiguous and out.shape == (nq, N)
+            if not isinstance(out, np.ndarray) or out.dtype != np.int32 or not out.flags.c_contiguous \
+                    or out.shape != (nq, N) or not out.flags.writeable:
+                raise ValueError(f"search: out must be a writeable C-contiguous int32 array of shape {(nq, N)}")
             optr = _vp(out)
         check(lib().sw_search(self.ptr, _vp(q_codes) if q_codes.size else None, _vp(q_offsets), nq, db.ptr,
                               _vp(matrix), int(gap_open), int(gap_extend), optr, _stream_ptr(stream)), self.ptr)
@@ -157,6 +192,24 @@ class Handle:
             raise ValueError("align: load the DB through Handle.load_db (sequence lengths needed)")
         return lens
 
+    def assembly(self, blocks, rows, cols, n_queries: int, n_cols: int) -> "Assembly":
+        """sw_assembly_create: blocks = int64[n][5] (src_off, row_off, col_off, n_rows, n_cols),
+        rows = int32 query indices, cols = int64 DB columns (caller order)."""
+        b = _host(blocks, np.int64).reshape(-1, 5)
+        rows = _host(rows, np.int32)
+        cols = _host(cols, np.int64)
+        tab = (Block * max(len(b), 1))()
+        for i, x in enumerate(b):
+            tab[i] = Block(*[int(v) for v in x])
+        out = ctypes.c_void_p()
+        check(lib().sw_assembly_create(self.ptr, ctypes.cast(tab, ctypes.c_void_p), len(b),
+                                       _vp(rows) if rows.size else None, len(rows),
+                                       _vp(cols) if cols.size else None, len(cols), int(n_queries), int(n_cols),
+                                       ctypes.byref(out)), self.ptr)
+        a = Assembly(self, out)
+        self._asm.append(a)
+        return a
+
     def last_stats(self) -> dict:
         s = Stats()
         check(lib().sw_last_stats(self.ptr, ctypes.byref(s)), self.ptr)
@@ -168,6 +221,8 @@ class Handle:
             self.ptr = None
             for d in self._dbs:
                 d.ptr = None
+            for a in self._asm:
+                a.ptr = None
 
     def __enter__(self):
         return self

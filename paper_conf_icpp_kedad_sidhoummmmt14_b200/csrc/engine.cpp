@@ -47,6 +47,8 @@ struct DevBuf {
   }
   cudaError_t ensure(size_t bytes) {
     if (bytes <= n && p) return cudaSuccess;
+    // growing: an earlier search (on any stream) may still use the old buffer
+    if (p) { cudaError_t e = cudaDeviceSynchronize(); if (e != cudaSuccess) return e; }
     release();
     size_t b = std::max<size_t>(bytes, 256);
     cudaError_t e = cudaMalloc(&p, b);
@@ -83,6 +85,7 @@ constexpr double CRIT_FRACTION = 0.35;  // pairs longer than this are launched s
 }  // namespace
 
 struct sw_db_s;
+struct sw_assembly_s;
 
 struct sw_handle_s {
   int device = 0;
@@ -90,14 +93,19 @@ struct sw_handle_s {
   uint32_t flags = 0;
   std::string err;
   std::vector<sw_db_s*> dbs;
+  std::vector<sw_assembly_s*> assemblies;
   // scratch (grown on demand)
   DevBuf qcodes, qoff, matrix, prof, bbuf, bbuf_long, counters, ovf, ovf_count, scores_tmp, rbuf, qdesc;
   DevBuf glinks, gflags;  // superstrip boundary rows and their counters (long pairs)
   DevBuf rgrows, rflags;  // re-score: CTA-to-CTA rows, counters
   DevBuf imap;            // short work item order
   DevBuf vq, sinfo;       // packed mode-1 slots: strip-padded query codes per half, per-strip info
-  int* pinned_count = nullptr;
   cudaEvent_t ev_begin = nullptr, ev_end = nullptr;
+  // the previous search's completion: a search on another stream waits for it on the
+  // device, because both use this handle's scratch
+  cudaEvent_t ev_done = nullptr;
+  cudaStream_t done_stream = nullptr;
+  bool done_valid = false;
   bool search_timed = false;
   bool timing_accumulate = false;
   std::vector<int> event_kind;
@@ -144,8 +152,15 @@ struct sw_db_s {
   // rows of out_n columns -- e.g. a rank's shard writing into rank 0's full matrix
   int64_t out_n = 0;
   bool mapped = false;
-  DevBuf dzero_cols;             // mapped: output columns of empty sequences (zeroed per search)
-  int64_t n_zero_cols = 0;
+  DevBuf dcols;                  // mapped: this DB's output columns, zeroed in every query row per search
+  int64_t n_cols = 0;
+};
+
+struct sw_assembly_s {
+  sw_handle_s* h = nullptr;
+  int n_blocks = 0;
+  int64_t total = 0, src_need = 0, n_queries = 0, N = 0;
+  DevBuf blocks, prefix, rows, cols;
 };
 
 static int32_t set_err(sw_handle_s* h, int32_t code, const std::string& m) {
@@ -456,13 +471,10 @@ int32_t sw_load_db_mapped(sw_handle_t h, const uint8_t* codes, const int64_t* of
     if (out_n > (int64_t(1) << 31) - 1) fail(SW_EUNSUPPORTED, "sw_load_db_mapped: out_n >= 2^31");
     if (!dp.empty())
       SW_CK(cudaMemcpyAsync(db->dpairs.p, dp.data(), dp.size() * sizeof(PairRec), cudaMemcpyHostToDevice, st));
-    std::vector<int64_t> zc;
-    for (int64_t d = 0; d < n_seqs; ++d)
-      if (db->seq_len[size_t(d)] == 0) zc.push_back(out_index[d]);
-    db->n_zero_cols = int64_t(zc.size());
-    if (!zc.empty()) {
-      SW_CK(db->dzero_cols.ensure(zc.size() * sizeof(int64_t)));
-      SW_CK(cudaMemcpyAsync(db->dzero_cols.p, zc.data(), zc.size() * sizeof(int64_t), cudaMemcpyHostToDevice, st));
+    db->n_cols = n_seqs;
+    if (n_seqs > 0) {
+      SW_CK(db->dcols.ensure(size_t(n_seqs) * sizeof(int64_t)));
+      SW_CK(cudaMemcpyAsync(db->dcols.p, out_index, size_t(n_seqs) * sizeof(int64_t), cudaMemcpyHostToDevice, st));
     }
     db->out_n = out_n;
     db->mapped = true;
@@ -947,6 +959,7 @@ int32_t sw_search(sw_handle_t h, const uint8_t* q_codes, const int64_t* q_offset
     const int alpha = db->alpha;
     SW_CK(cudaSetDevice(h->device));
     cudaStream_t st = reinterpret_cast<cudaStream_t>(cuda_stream);
+    if (h->done_valid && h->done_stream != st) SW_CK(cudaStreamWaitEvent(st, h->ev_done, 0));
     h->stats = sw_stats_t{};
     if (!h->timing_accumulate) h->n_events_used = 0;
     h->last_stream = st;
@@ -971,7 +984,9 @@ int32_t sw_search(sw_handle_t h, const uint8_t* q_codes, const int64_t* q_offset
     for (int i = 0; i < alpha * alpha; ++i) smax = std::max<int>(smax, matrix[i]);
     // int16 re-score threshold: flag if max >= 32767 - S_max
     int32_t thr = smax > 0 ? 32767 - smax : 32768;
-    if (h->opt_thr > 0) thr = int32_t(h->opt_thr);
+    // a forced threshold may only be lower: above 32767 - S_max a wrapped int16
+    // value could pass unflagged
+    if (h->opt_thr > 0) thr = int32_t(std::min<int64_t>(h->opt_thr, thr));
     // output
     cudaPointerAttributes pa{};
     bool dev_scores = false;
@@ -1004,14 +1019,14 @@ int32_t sw_search(sw_handle_t h, const uint8_t* q_codes, const int64_t* q_offset
     int launches = 0;
     if (!db->mapped) {
       SW_CK(cudaMemsetAsync(dscores, 0, out_bytes, st));
-    } else if (db->n_zero_cols > 0) {  // only this DB's columns: other ranks write the rest
-      SW_CK(launch_zero_columns(dscores, N, n_queries, db->dzero_cols.as<int64_t>(), db->n_zero_cols, st));
+    } else if (db->n_cols > 0) {  // only this DB's columns (other ranks / shards own the rest)
+      SW_CK(launch_zero_columns(dscores, N, n_queries, db->dcols.as<int64_t>(), db->n_cols, st));
       ++launches;
     }
     // overflow list capacity: a pair can only be flagged if min(m, n) * S_max >= thr
     int64_t ovf_cap = 0;
     if (smax > 0) {
-      const int64_t need = (int64_t(thr) + smax - 1) / smax;  // min length that can reach thr
+      const int64_t need = std::max<int64_t>(1, (int64_t(thr) + smax - 1) / smax);  // min length that can reach thr
       // sorted_lens is descending: count the DB sequences of length >= need
       const int64_t nd_ge = std::lower_bound(db->sorted_lens.begin(), db->sorted_lens.end(), need,
                                              [](int64_t v, int64_t x) { return v >= x; }) -
@@ -1046,59 +1061,60 @@ int32_t sw_search(sw_handle_t h, const uint8_t* q_codes, const int64_t* q_offset
     const uint8_t* dq = h->qcodes.as<uint8_t>();
     launch_all(lc, qlen, qoff0, cells_computed, launches);
     if (ovf_cap > 0) {
-      // the flagged list is usually empty or tiny: read its length (one sync,
-      // only for searches whose bounds allow an int16 overflow at all)
-      if (!h->pinned_count) SW_CK(cudaMallocHost(&h->pinned_count, sizeof(int)));
-      SW_CK(cudaMemcpyAsync(h->pinned_count, h->ovf_count.p, sizeof(int), cudaMemcpyDeviceToHost, st));
-      SW_CK(cudaStreamSynchronize(st));
-      const int cnt = int(std::min<int64_t>(*h->pinned_count, ovf_cap));
-      if (cnt > 0) {
-        const int32_t Lmax = std::max(max_short, max_long);
-        int64_t mmax = 1;
-        for (auto L : qlen) mmax = std::max(mmax, L);
-        const int rows_per_strip = 32 * RESCORE_R;
-        const int nstrips = int((mmax + rows_per_strip - 1) / rows_per_strip);
-        // one strip per warp (a single round): CTA c only waits on CTA c-1,
-        // which took its item earlier, so any grid size is deadlock-free and
-        // the pair's critical path is its columns + strips x (32 + lag)
-        const int K = std::max(1, (nstrips + RESCORE_WARPS - 1) / RESCORE_WARPS);
-        const int grid = std::max(1, std::min<int>(cnt * K, h->sms * 4));
-        const int bcap = Lmax + 32 + 72;
-        SW_CK(h->rbuf.ensure(size_t(grid) * RESCORE_WARPS * bcap * sizeof(int2)));
-        SW_CK(h->rgrows.ensure(size_t(cnt) * K * bcap * sizeof(int2) + 16));
-        const size_t nint = size_t(cnt) * K + 2 * size_t(cnt) + 1;
-        SW_CK(h->rflags.ensure(nint * sizeof(int)));
-        SW_CK(cudaMemsetAsync(h->rflags.p, 0, nint * sizeof(int), st));
-        int* fl = h->rflags.as<int>();
-        RescoreArgs r{};
-        r.qcodes = dq;
-        r.qoff = h->qoff.as<int64_t>();
-        r.stream = db->stream.as<uint16_t>();
-        r.pairs = db->dpairs.as<PairRec>();
-        r.matrix = h->matrix.as<int8_t>();
-        r.alpha = alpha;
-        r.ovf = h->ovf.as<OvfRec>();
-        r.n_entries = cnt;
-        r.K = K;
-        r.gflags = fl;
-        r.acc = fl + size_t(cnt) * K;
-        r.done = r.acc + cnt;
-        r.work_counter = r.done + cnt;
-        r.bbuf = h->rbuf.as<int2>();
-        r.grows = h->rgrows.as<int2>();
-        r.bcap = bcap;
-        r.scores = dscores;
-        r.n_seqs = N;
-        r.Gs = gap_open;
-        r.Ge = gap_extend;
-        SW_CK(launch_rescore(grid, r, st));
-        ++launches;
-      }
+      // Exact int32 re-score of the flagged pairs, enqueued unconditionally: the
+      // kernel reads the flagged count on the device and exits at once when it is
+      // zero, so the host never waits for the scoring kernel (stream-ordered).
+      const int32_t Lmax = std::max(max_short, max_long);
+      int64_t mmax = 1;
+      for (auto L : qlen) mmax = std::max(mmax, L);
+      const int rows_per_strip = 32 * RESCORE_R;
+      const int nstrips = int((mmax + rows_per_strip - 1) / rows_per_strip);
+      // one round of RESCORE_WARPS strips per CTA (every wait targets an earlier item)
+      const int K = std::max(1, (nstrips + RESCORE_WARPS - 1) / RESCORE_WARPS);
+      const int grid = int(std::max<int64_t>(1, std::min<int64_t>(ovf_cap * K, 2 * h->sms)));
+      const int ne_slots = int(std::min<int64_t>(ovf_cap, 64));
+      const int bcap = Lmax + 32 + 72;
+      SW_CK(h->rbuf.ensure(size_t(grid) * RESCORE_WARPS * bcap * sizeof(int2)));
+      SW_CK(h->rgrows.ensure(size_t(ne_slots) * K * bcap * sizeof(int2) + 16));
+      const size_t nflag_b = size_t(ne_slots) * K * sizeof(unsigned long long);
+      const size_t nint = 2 * size_t(ovf_cap) + 1;
+      SW_CK(h->rflags.ensure(nflag_b + nint * sizeof(int)));
+      SW_CK(cudaMemsetAsync(h->rflags.p, 0, nflag_b + nint * sizeof(int), st));
+      int* fl = reinterpret_cast<int*>(h->rflags.as<uint8_t>() + nflag_b);
+      RescoreArgs r{};
+      r.qcodes = dq;
+      r.qoff = h->qoff.as<int64_t>();
+      r.stream = db->stream.as<uint16_t>();
+      r.pairs = db->dpairs.as<PairRec>();
+      r.matrix = h->matrix.as<int8_t>();
+      r.alpha = alpha;
+      r.ovf = h->ovf.as<OvfRec>();
+      r.ovf_count = h->ovf_count.as<int>();
+      r.ovf_cap = int(ovf_cap);
+      r.K = K;
+      r.ne_slots = ne_slots;
+      r.gflags = h->rflags.as<unsigned long long>();
+      r.acc = fl;
+      r.done = r.acc + ovf_cap;
+      r.work_counter = r.done + ovf_cap;
+      r.bbuf = h->rbuf.as<int2>();
+      r.grows = h->rgrows.as<int2>();
+      r.bcap = bcap;
+      r.scores = dscores;
+      r.n_seqs = N;
+      r.Gs = gap_open;
+      r.Ge = gap_extend;
+      SW_CK(launch_rescore(grid, r, st));
+      ++launches;
     }
     if (timing) {
       SW_CK(cudaEventRecord(h->ev_end, st));
       h->search_timed = true;
     }
+    if (!h->ev_done) SW_CK(cudaEventCreateWithFlags(&h->ev_done, cudaEventDisableTiming));
+    SW_CK(cudaEventRecord(h->ev_done, st));
+    h->done_stream = st;
+    h->done_valid = true;
     if (!dev_scores) {
       SW_CK(cudaMemcpyAsync(scores, dscores, out_bytes, cudaMemcpyDeviceToHost, st));
       SW_CK(cudaStreamSynchronize(st));
@@ -1304,6 +1320,88 @@ int32_t sw_align(sw_handle_t h, const uint8_t* q_codes, const int64_t* q_offsets
   });
 }
 
+// ----------------------------------------------------------------------------
+// Merge of gathered score blocks.
+int32_t sw_assembly_create(sw_handle_t h, const sw_block_t* blocks, int32_t n_blocks, const int32_t* rows,
+                           int64_t n_rows, const int64_t* cols, int64_t n_cols, int32_t n_queries, int64_t N,
+                           sw_assembly_t* out) {
+  if (!h) return set_err(nullptr, SW_EINVAL, "sw_assembly_create: handle is NULL");
+  if (!out) return set_err(h, SW_EINVAL, "sw_assembly_create: out is NULL");
+  *out = nullptr;
+  sw_assembly_s* a = nullptr;
+  int32_t rc = guarded(h, [&] {
+    if (n_blocks < 0 || n_rows < 0 || n_cols < 0 || n_queries < 0 || N < 0)
+      fail(SW_EINVAL, "sw_assembly_create: negative size");
+    if ((n_blocks > 0 && !blocks) || (n_rows > 0 && !rows) || (n_cols > 0 && !cols))
+      fail(SW_EINVAL, "sw_assembly_create: NULL table");
+    for (int64_t i = 0; i < n_rows; ++i)
+      if (rows[i] < 0 || rows[i] >= n_queries) fail(SW_EINVAL, "sw_assembly_create: query index out of range");
+    for (int64_t i = 0; i < n_cols; ++i)
+      if (cols[i] < 0 || cols[i] >= N) fail(SW_EINVAL, "sw_assembly_create: column out of range");
+    std::vector<AsmBlock> bk(static_cast<size_t>(n_blocks));
+    std::vector<int64_t> prefix(size_t(n_blocks) + 1, 0);
+    int64_t need = 0;
+    for (int b = 0; b < n_blocks; ++b) {
+      const sw_block_t& x = blocks[b];
+      if (x.n_rows < 0 || x.n_cols < 0 || x.src_off < 0 || x.row_off < 0 || x.col_off < 0 ||
+          x.row_off + x.n_rows > n_rows || x.col_off + x.n_cols > n_cols)
+        fail(SW_EINVAL, "sw_assembly_create: block " + std::to_string(b) + " out of range");
+      bk[size_t(b)] = AsmBlock{x.src_off, x.row_off, x.col_off, x.n_rows, x.n_cols};
+      prefix[size_t(b) + 1] = prefix[size_t(b)] + x.n_rows * x.n_cols;
+      need = std::max(need, x.src_off + x.n_rows * x.n_cols);
+    }
+    SW_CK(cudaSetDevice(h->device));
+    a = new sw_assembly_s();
+    a->h = h;
+    a->n_blocks = n_blocks;
+    a->total = prefix.back();
+    a->src_need = need;
+    a->n_queries = n_queries;
+    a->N = N;
+    SW_CK(a->blocks.ensure(std::max<size_t>(bk.size(), 1) * sizeof(AsmBlock)));
+    SW_CK(a->prefix.ensure(prefix.size() * sizeof(int64_t)));
+    SW_CK(a->rows.ensure(size_t(std::max<int64_t>(n_rows, 1)) * sizeof(int32_t)));
+    SW_CK(a->cols.ensure(size_t(std::max<int64_t>(n_cols, 1)) * sizeof(int64_t)));
+    if (n_blocks) SW_CK(cudaMemcpy(a->blocks.p, bk.data(), bk.size() * sizeof(AsmBlock), cudaMemcpyHostToDevice));
+    SW_CK(cudaMemcpy(a->prefix.p, prefix.data(), prefix.size() * sizeof(int64_t), cudaMemcpyHostToDevice));
+    if (n_rows) SW_CK(cudaMemcpy(a->rows.p, rows, size_t(n_rows) * sizeof(int32_t), cudaMemcpyHostToDevice));
+    if (n_cols) SW_CK(cudaMemcpy(a->cols.p, cols, size_t(n_cols) * sizeof(int64_t), cudaMemcpyHostToDevice));
+  });
+  if (rc != SW_OK) {
+    delete a;
+    return rc;
+  }
+  h->assemblies.push_back(a);
+  *out = a;
+  return SW_OK;
+}
+
+int32_t sw_assemble(sw_assembly_t a, const int32_t* src, int64_t src_len, int32_t* out, void* cuda_stream) {
+  if (!a || !a->h) return set_err(nullptr, SW_EINVAL, "sw_assemble: assembly is NULL");
+  sw_handle_s* h = a->h;
+  return guarded(h, [&] {
+    if (src_len < a->src_need) fail(SW_EINVAL, "sw_assemble: src shorter than the blocks");
+    if (a->total == 0) return;
+    if (!src || !out) fail(SW_EINVAL, "sw_assemble: NULL buffer");
+    SW_CK(cudaSetDevice(h->device));
+    SW_CK(launch_assemble(src, a->blocks.as<AsmBlock>(), a->n_blocks, a->prefix.as<int64_t>(), a->total,
+                          a->rows.as<int32_t>(), a->cols.as<int64_t>(), out, a->N, h->sms,
+                          reinterpret_cast<cudaStream_t>(cuda_stream)));
+  });
+}
+
+int32_t sw_assembly_free(sw_assembly_t a) {
+  if (!a) return SW_OK;
+  if (a->h) {
+    cudaSetDevice(a->h->device);
+    auto& v = a->h->assemblies;
+    auto it = std::find(v.begin(), v.end(), a);
+    if (it != v.end()) v.erase(it);
+  }
+  delete a;
+  return SW_OK;
+}
+
 int32_t sw_last_stats(sw_handle_t h, sw_stats_t* out) {
   if (!h || !out) return set_err(h, SW_EINVAL, "sw_last_stats: NULL argument");
   return guarded(h, [&] {
@@ -1354,13 +1452,15 @@ int32_t sw_free(sw_handle_t h) {
     delete db;
   }
   h->dbs.clear();
+  for (auto* a : h->assemblies) delete a;
+  h->assemblies.clear();
   for (auto& e : h->events) {
     cudaEventDestroy(e.first);
     cudaEventDestroy(e.second);
   }
   for (cudaEvent_t e : {h->ev_begin, h->ev_end})
     if (e) cudaEventDestroy(e);
-  if (h->pinned_count) cudaFreeHost(h->pinned_count);
+  if (h->ev_done) cudaEventDestroy(h->ev_done);
   delete h;
   return SW_OK;
 }

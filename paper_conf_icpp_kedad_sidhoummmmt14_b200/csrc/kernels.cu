@@ -739,11 +739,26 @@ cudaError_t launch_inter(int G, int R, int NT, int grid, int smem_bytes, const I
 // ---------------------------------------------------------------------------
 // Exact int32 re-score of flagged pairs.  The same chained
 // wavefront as the long-pair mode, one problem per lane in int32 (s32 DPX),
-// S read from a shared 33x33 matrix: a flagged pair is split over K CTAs,
-// strips dealt round-robin (round r of CTA c = strips W*(K*r + c) .. +W-1,
-// 32 lanes x RESCORE_R rows each), chained warp to warp through per-CTA link
-// rows + shared counters and CTA to CTA through global rows + GPU-scope
-// counters.  The CTAs' maxima meet in acc[e]; the last CTA writes the score.
+// S read from a shared 33x33 matrix.  A flagged pair (entry) is split over K
+// CTAs, one round each: CTA c of entry e holds strips W*c .. W*c + W-1 (32
+// lanes x RESCORE_R rows each), chained warp to warp through per-CTA link rows
+// + shared counters and CTA c-1 -> c through a global row + GPU-scope counter.
+// Every wait targets an item taken earlier (CTA c-1 of the same entry, or the
+// last users of a reused row block), so any grid size and any co-residency is
+// deadlock-free.  The number of entries is read here, on the device: the host
+// enqueues this kernel unconditionally and never waits for the scoring kernel.
+// Row blocks are reused: entry e uses block e % ne_slots, after the ne_slots-
+// earlier entry's K CTAs are done; counters carry (entry + 1) in their high
+// word, so a stale value of the block's previous entry never satisfies a wait.
+__device__ __forceinline__ unsigned long long ld_acquire_gpu_u64(const unsigned long long* p) {
+  unsigned long long v;
+  asm volatile("ld.acquire.gpu.global.b64 %0, [%1];" : "=l"(v) : "l"(p) : "memory");
+  return v;
+}
+__device__ __forceinline__ void st_release_gpu_u64(unsigned long long* p, unsigned long long v) {
+  asm volatile("st.release.gpu.global.b64 [%0], %1;" :: "l"(p), "l"(v) : "memory");
+}
+
 __global__ void __launch_bounds__(RESCORE_WARPS * 32) rescore_kernel(RescoreArgs a) {
   constexpr int R = RESCORE_R;
   constexpr int W = RESCORE_WARPS;
@@ -760,7 +775,8 @@ __global__ void __launch_bounds__(RESCORE_WARPS * 32) rescore_kernel(RescoreArgs
   const bool lead = lane == 0, tail = lane == 31;
   int2* __restrict__ links = a.bbuf + (size_t)blockIdx.x * W * a.bcap;
   const int K = a.K;
-  const int n_items = a.n_entries * K;
+  const int n_entries = min(*(volatile const int*)a.ovf_count, a.ovf_cap);
+  const int n_items = n_entries * K;
   const int pad = a.alpha;
   const int nGe = -a.Ge, nGsGe = -(a.Gs + a.Ge);
   for (;;) {
@@ -781,37 +797,45 @@ __global__ void __launch_bounds__(RESCORE_WARPS * 32) rescore_kernel(RescoreArgs
     const int T = L + 32;
     const uint2* __restrict__ codes = reinterpret_cast<const uint2*>(a.stream + pr.off);
     const uint32_t padw = uint32_t(pad) * 0x01010101u;
-    int2* grow = a.grows + (int64_t)e * K * a.bcap;
-    int* gflag = a.gflags + (int64_t)e * K;
+    const int blk = e % a.ne_slots;
+    int2* grow = a.grows + (int64_t)blk * K * a.bcap;
+    unsigned long long* gflag = a.gflags + (int64_t)blk * K;
+    const unsigned long long gen = (unsigned long long)(e + 1) << 32;
     const int j = W - 1 - warp;  // producers on higher warp ids (see inter_kernel)
+    const int s = W * c + j;
+    // the block's previous entry must be finished before this CTA writes its row
+    if (c + 1 < K && e >= a.ne_slots && warp == 0) {
+      if (lane == 0)
+        while (atomicAdd(a.done + (e - a.ne_slots), 0) < K) __nanosleep(256);
+      __syncwarp();
+    }
+    __syncthreads();
     int best = 0;
-    for (int r = 0;; ++r) {
-      const int s = W * (K * r + c) + j;
-      if (s >= nstrips) break;
+    if (s < nstrips) {
       const bool rd = s > 0, wr = s + 1 < nstrips;
-      Link lk{};
-      const int2* rp;
-      int2* wp;
-      if (j > 0 || K == 1) {
-        const int jl = (j + W - 1) % W;
-        rp = links + (size_t)jl * a.bcap;
-        lk.in = &s_prog[jl];
-      } else {
-        const int pc = (c + K - 1) % K;
-        rp = grow + (int64_t)pc * a.bcap;
-        lk.in = gflag + pc;
-        lk.in_gpu = true;
-      }
-      lk.in_base = (s - 1) << 20;
-      if (j < W - 1 || K == 1) {
-        wp = links + (size_t)j * a.bcap;
-        lk.out = &s_prog[j];
-      } else {
-        wp = grow + (int64_t)c * a.bcap;
-        lk.out = gflag + c;
-        lk.out_gpu = true;
-      }
-      lk.out_base = s << 20;
+      const bool in_gpu = (j == 0 && c > 0), out_gpu = (j == W - 1 && c + 1 < K);
+      const int2* rp = in_gpu ? grow + (int64_t)(c - 1) * a.bcap : links + (size_t)(j > 0 ? j - 1 : 0) * a.bcap;
+      int2* wp = out_gpu ? grow + (int64_t)c * a.bcap : links + (size_t)j * a.bcap;
+      const int in_base = (s - 1) << 20, out_base = s << 20;
+      int seen = -1;
+      auto wait_in = [&](int need) {
+        if (seen >= need) return;
+        for (;;) {
+          int v = 0;
+          if (lead) {
+            if (in_gpu) {
+              const unsigned long long x = ld_acquire_gpu_u64(gflag + (c - 1));
+              v = (x >> 32) == (unsigned long long)(e + 1) ? int(x & 0xffffffffu) : -1;
+            } else {
+              v = ld_acquire_cta(&s_prog[j - 1]);
+            }
+          }
+          v = __shfl_sync(FULL, v, 0);
+          if (v >= need) { seen = v; break; }
+          __nanosleep(in_gpu ? 256 : 64);
+        }
+        if (in_gpu) __threadfence();
+      };
       rp += 31;
       int qr[R], Hl[R], E[R];
 #pragma unroll
@@ -825,8 +849,7 @@ __global__ void __launch_bounds__(RESCORE_WARPS * 32) rescore_kernel(RescoreArgs
       const int2 z2 = make_int2(0, 0);
       uint2 cw = make_uint2(padw, padw);
       int2 tb0 = z2, tb1 = z2, tb2 = z2, tb3 = z2;
-      int seen = -1;
-      if (rd && L > 0) wait_progress(lk, lk.in_base + min(4 + 31 + RESCORE_LAG, L + 32), seen);
+      if (rd && L > 0) wait_in(in_base + min(4 + 31 + RESCORE_LAG, L + 32));
       if (lead && L > 0) {
         cw = codes[0];
         if (rd) { tb0 = __ldcg(rp + 0); tb1 = __ldcg(rp + 1); tb2 = __ldcg(rp + 2); tb3 = __ldcg(rp + 3); }
@@ -835,7 +858,7 @@ __global__ void __launch_bounds__(RESCORE_WARPS * 32) rescore_kernel(RescoreArgs
       for (int t0 = 0; t0 < T; t0 += 4) {
         const uint2 cwc = cw;
         const int2 c0 = tb0, c1 = tb1, c2 = tb2, c3 = tb3;
-        if (rd && t0 + 4 < L) wait_progress(lk, lk.in_base + min(t0 + 8 + 31 + RESCORE_LAG, L + 32), seen);
+        if (rd && t0 + 4 < L) wait_in(in_base + min(t0 + 8 + 31 + RESCORE_LAG, L + 32));
         if (lead) {
           if (t0 + 4 < L) {
             cw = codes[(t0 + 4) >> 2];
@@ -882,8 +905,9 @@ __global__ void __launch_bounds__(RESCORE_WARPS * 32) rescore_kernel(RescoreArgs
           if (wr && tail) __stcg(wp + t0 + jj, make_int2(sH, sF));
         }
         if (wr && tail) {
-          if (!lk.out_gpu) st_release_cta(lk.out, lk.out_base + t0 + 4);
-          else if (((t0 >> 2) & 3) == 3 || t0 + 4 >= T) st_release_gpu(lk.out, lk.out_base + t0 + 4);
+          if (!out_gpu) st_release_cta(&s_prog[j], out_base + t0 + 4);
+          else if (((t0 >> 2) & 3) == 3 || t0 + 4 >= T)
+            st_release_gpu_u64(gflag + c, gen | (unsigned long long)(unsigned)(out_base + t0 + 4));
         }
       }
     }
@@ -897,6 +921,7 @@ __global__ void __launch_bounds__(RESCORE_WARPS * 32) rescore_kernel(RescoreArgs
       const int id = o.half ? pr.id1 : pr.id0;
       if (K == 1) {
         a.scores[(int64_t)o.q * a.n_seqs + id] = b;
+        atomicAdd(a.done + e, 1);
       } else {
         atomicMax(a.acc + e, b);
         __threadfence();
@@ -927,6 +952,37 @@ cudaError_t launch_zero_columns(int32_t* scores, int64_t stride, int nq, const i
   const int64_t n = int64_t(nq) * ncols;
   if (n <= 0) return cudaSuccess;
   zero_columns_kernel<<<int(std::min<int64_t>((n + 255) / 256, 1024)), 256, 0, st>>>(scores, stride, nq, cols, ncols);
+  return cudaGetLastError();
+}
+
+// Merge of gathered score blocks into scores[Q][N] in the caller's order (SURVEY
+// 8(a) a8; the master's "merge").  Block b holds rows x cols
+// int32 values at src + src_off (row-major), row i -> query rows[row_off + i],
+// column k -> DB column cols[col_off + k].  One thread per element, grid-stride
+// over a flat index; a small per-block prefix table locates the block.
+__global__ void assemble_kernel(const int32_t* __restrict__ src, const AsmBlock* __restrict__ blocks, int n_blocks,
+                                const int64_t* __restrict__ prefix, const int32_t* __restrict__ rows,
+                                const int64_t* __restrict__ cols, int32_t* __restrict__ out, int64_t N) {
+  const int64_t total = prefix[n_blocks];
+  for (int64_t x = blockIdx.x * int64_t(blockDim.x) + threadIdx.x; x < total; x += int64_t(gridDim.x) * blockDim.x) {
+    int lo = 0, hi = n_blocks - 1;  // the block holding element x: prefix[b] <= x < prefix[b+1]
+    while (lo < hi) {
+      const int mid = (lo + hi + 1) >> 1;
+      if (prefix[mid] <= x) lo = mid; else hi = mid - 1;
+    }
+    const AsmBlock bk = blocks[lo];
+    const int64_t e = x - prefix[lo];
+    const int64_t i = e / bk.n_cols, k = e - i * bk.n_cols;
+    out[int64_t(rows[bk.row_off + i]) * N + cols[bk.col_off + k]] = src[bk.src_off + e];
+  }
+}
+
+cudaError_t launch_assemble(const int32_t* src, const AsmBlock* blocks, int n_blocks, const int64_t* prefix,
+                            int64_t total, const int32_t* rows, const int64_t* cols, int32_t* out, int64_t N,
+                            int sms, cudaStream_t st) {
+  if (total <= 0) return cudaSuccess;
+  const int grid = int(std::min<int64_t>((total + 255) / 256, int64_t(sms) * 8));
+  assemble_kernel<<<grid, 256, 0, st>>>(src, blocks, n_blocks, prefix, rows, cols, out, N);
   return cudaGetLastError();
 }
 

@@ -16,6 +16,7 @@
 //   Binary search on lambda between Bmin and Bmax (L468-481, reading S-5).
 // With m = 0 CPUs (the B200 box, reading S-6) every task is a GPU task and the
 // method reduces to binary search + LPT list scheduling.
+#include <new>
 #include <algorithm>
 #include <cmath>
 #include <limits>
@@ -204,15 +205,29 @@ int32_t binary_search(step_fn step, int64_t n_tasks, const double* p_cpu, const 
 }
 }  // namespace
 
+// No C++ exception may cross the C ABI: a failed host allocation becomes SW_ENOMEM.
+static int32_t guarded_search(step_fn step, int64_t n_tasks, const double* p_cpu, const double* p_gpu,
+                              int32_t n_cpu, int32_t n_gpu, int32_t* out_pe, double* out_makespan,
+                              double* out_lambda) {
+  try {
+    return binary_search(step, n_tasks, p_cpu, p_gpu, n_cpu, n_gpu, out_pe, out_makespan, out_lambda);
+  } catch (const std::bad_alloc&) {
+    return SW_ENOMEM;
+  } catch (...) {
+    return SW_EINVAL;
+  }
+}
+
 extern "C" int32_t sw_schedule_dual(int64_t n_tasks, const double* p_cpu, const double* p_gpu, int32_t n_cpu,
                                     int32_t n_gpu, int32_t* out_pe, double* out_makespan, double* out_lambda) {
-  return binary_search(dual_step, n_tasks, p_cpu, p_gpu, n_cpu, n_gpu, out_pe, out_makespan, out_lambda);
+  return guarded_search(dual_step, n_tasks, p_cpu, p_gpu, n_cpu, n_gpu, out_pe, out_makespan, out_lambda);
 }
 
 extern "C" int32_t sw_schedule_dual_dp(int64_t n_tasks, const double* p_cpu, const double* p_gpu, int32_t n_cpu,
                                        int32_t n_gpu, int32_t* out_pe, double* out_makespan, double* out_lambda) {
   // the DP table holds (m+1)(k+1)(4kn+1) states per task
   const double states = double(n_cpu + 1) * double(n_gpu + 1) * (4.0 * double(n_gpu) * double(n_tasks) + 1.0);
-  if (n_tasks > 0 && states * double(n_tasks) > 4.0e9) return SW_EUNSUPPORTED;
-  return binary_search(dual_step_dp, n_tasks, p_cpu, p_gpu, n_cpu, n_gpu, out_pe, out_makespan, out_lambda);
+  // (one byte of choice table per state and task, rebuilt per bisection step: <= 256 MB)
+  if (n_tasks > 0 && states * double(n_tasks) > 2.56e8) return SW_EUNSUPPORTED;
+  return guarded_search(dual_step_dp, n_tasks, p_cpu, p_gpu, n_cpu, n_gpu, out_pe, out_makespan, out_lambda);
 }

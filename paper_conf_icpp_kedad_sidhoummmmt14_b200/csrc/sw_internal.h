@@ -162,18 +162,28 @@ struct RescoreArgs {
   const int8_t* matrix;      // alpha x alpha
   int alpha;
   const OvfRec* ovf;         // flagged pairs
-  int n_entries;             // number of flagged pairs (host-read count)
-  int K;                     // CTAs per flagged pair
+  const int* ovf_count;      // device: flagged pairs written by the scoring kernel (read on the device,
+  int ovf_cap;               //   so the host never waits for it); entries = min(*ovf_count, ovf_cap)
+  int K;                     // CTAs per flagged pair (one round of RESCORE_WARPS strips each)
+  int ne_slots;              // CTA-to-CTA row blocks: entry e uses block e % ne_slots
   int* work_counter;         // zeroed
-  int2* bbuf;                // per-CTA link rows, [gridDim][RESCORE_WARPS][bcap]
-  int2* grows;               // CTA-to-CTA rows, [n_entries][K][bcap]
-  int* gflags;               // [n_entries][K], zeroed
-  int* acc;                  // [n_entries] partial maxima, zeroed
-  int* done;                 // [n_entries] finished CTAs, zeroed
+  int2* bbuf;                // per-CTA warp link rows, [gridDim][RESCORE_WARPS][bcap]
+  int2* grows;               // CTA-to-CTA rows, [ne_slots][K][bcap]
+  unsigned long long* gflags;  // [ne_slots][K]: (entry + 1) << 32 | progress (generation-tagged), zeroed
+  int* acc;                  // [ovf_cap] partial maxima, zeroed
+  int* done;                 // [ovf_cap] finished CTAs per entry, zeroed
   int bcap;
   int32_t* scores;           // [nq][n_seqs]
   int64_t n_seqs;
   int32_t Gs, Ge;
+};
+
+// One gathered score block (sw_assemble): rows x cols int32 at src + src_off.
+struct AsmBlock {
+  int64_t src_off;   // elements
+  int64_t row_off;   // into the rows table (query indices)
+  int64_t col_off;   // into the cols table (DB columns)
+  int64_t n_rows, n_cols;
 };
 
 // kernels.cu entry points (host side launchers); return cudaError_t
@@ -193,6 +203,9 @@ cudaError_t launch_rescore(int grid, const RescoreArgs& a, cudaStream_t st);
 // scores[q * stride + cols[c]] = 0 for every query q < nq and column c < ncols
 cudaError_t launch_zero_columns(int32_t* scores, int64_t stride, int nq, const int64_t* cols, int64_t ncols,
                                 cudaStream_t st);
+cudaError_t launch_assemble(const int32_t* src, const AsmBlock* blocks, int n_blocks, const int64_t* prefix,
+                            int64_t total, const int32_t* rows, const int64_t* cols, int32_t* out, int64_t N,
+                            int sms, cudaStream_t st);
 constexpr int RESCORE_WARPS = 8;
 constexpr int RESCORE_R = 8;
 

@@ -66,10 +66,29 @@ class Plan:
     by_gpu: dict = field(default_factory=dict)  # gpu -> {shard: [queries]}
 
 
-def place(q_lens, shards, shard_residues, n_gpus: int, rate: float = 1.0) -> Plan:
+# GPU time model of one (query, shard) task on a B200 (p_j from a
+# calibrated rate).  The scoring kernel sweeps whole strips of STRIP_ROWS query
+# rows (the geometry chosen for Swiss-Prot-like DBs), so a query of m residues
+# costs ceil(m / STRIP_ROWS) * STRIP_ROWS rows -- which is why short queries run
+# at a lower cell rate (the per-query rates measured in
+# profiles/r01_hybrid_probe.jsonl: 144 aa ~0.75 of the long-query rate); plus a
+# per-task share of the launch and its tail.  RATE: the long-query cell rate of
+# the C3 bench (profiles/r01_end_bench_c3.json).
+STRIP_ROWS = 96
+RATE = 6.9e12          # computed cells per second per B200
+T_TASK = 5.0e-5        # seconds per task (profile build, launch tail share)
+
+
+def gpu_task_time(m: int, residues: float) -> float:
+    rows = -(-int(m) // STRIP_ROWS) * STRIP_ROWS if m > 0 else 0
+    return rows * float(residues) / RATE + (T_TASK if m > 0 and residues > 0 else 0.0)
+
+
+def place(q_lens, shards, shard_residues, n_gpus: int, rate: float | None = None) -> Plan:
     """Dual-approximation placement of (query, shard) tasks on n_gpus GPUs.
 
-    p_gpu(q, s) = m_q * residues(s) / rate  -- cells over a calibrated cell rate.
+    p_gpu(q, s) = gpu_task_time(m_q, residues(s)) (calibrated model), or
+    m_q * residues(s) / rate when a plain cell rate is given.
     """
     q_lens = [int(x) for x in q_lens]
     tasks = [(q, s) for q in range(len(q_lens)) for s in range(len(shards))]
@@ -77,7 +96,10 @@ def place(q_lens, shards, shard_residues, n_gpus: int, rate: float = 1.0) -> Pla
 
 
 def _place(q_lens, shards, n_gpus, rate, tasks, res) -> Plan:
-    p_gpu = np.array([q_lens[q] * res[s] / rate for q, s in tasks], dtype=np.float64)
+    if rate is None:
+        p_gpu = np.array([gpu_task_time(q_lens[q], res[s]) for q, s in tasks], dtype=np.float64)
+    else:
+        p_gpu = np.array([q_lens[q] * res[s] / rate for q, s in tasks], dtype=np.float64)
     p_cpu = p_gpu * 1e6  # no CPU PEs on the B200 box (m = 0); unused when n_cpu = 0
     if len(tasks):
         pe, mk, lam = schedule_dual(p_cpu, p_gpu, 0, n_gpus)
@@ -113,6 +135,119 @@ def assemble(plan: Plan, n_queries: int, n_seqs: int, flats) -> np.ndarray:
             pos += len(qs) * len(idx)
             out[np.ix_(qs, idx)] = blk
     return out
+
+
+def assembly_tables(plan: Plan):
+    """Block tables of the gathered buffer for sw_assemble (every rank's flat block
+    list, rank r's at offset r * cap, cap = the largest rank's flat size):
+    (blocks int64[n][5] = src_off, row_off, col_off, n_rows, n_cols; rows int32;
+    cols int64; cap).  A shard's column list is stored once."""
+    world = plan.n_gpus
+    cap = max([flat_size(plan, r) for r in range(world)] + [1])
+    blocks, rows, cols, col_off = [], [], [], {}
+    n_rows = 0
+    n_cols = 0
+    for r in range(world):
+        pos = r * cap
+        for s, qs in local_blocks(plan, r):
+            idx = plan.shards[s]
+            if s not in col_off:
+                col_off[s] = n_cols
+                cols.append(np.asarray(idx, dtype=np.int64))
+                n_cols += len(idx)
+            blocks.append((pos, n_rows, col_off[s], len(qs), len(idx)))
+            rows.append(np.asarray(qs, dtype=np.int32))
+            n_rows += len(qs)
+            pos += len(qs) * len(idx)
+    cat = lambda xs, dt: np.concatenate(xs).astype(dt) if xs else np.zeros(0, dt)  # noqa: E731
+    return (np.array(blocks, dtype=np.int64).reshape(-1, 5), cat(rows, np.int32), cat(cols, np.int64), cap)
+
+
+class ShardedSearch:
+    """One rank's part of the multi-GPU search; bench.py and the
+    tests run THIS code path.
+
+    Setup (untimed, like a resident search service): the DB is cut into
+    n_shards snake-dealt shards (default 4 per GPU), the (query, shard) tasks are
+    placed by the dual approximation (sw_schedule_dual, calibrated task times),
+    this rank loads the shards its tasks reference and prepares one sw_search
+    per (shard, query list) block into a flat device buffer.
+    step(): the rank's searches, then -- the single data-path exchange -- the
+    all-gather of the flat blocks (NCCL over NVLink; gloo with host staging for
+    functional runs), then on rank 0 sw_assemble merges them into scores[Q][N]
+    in the caller's order (the master's merge).  With one
+    GPU and one shard the search writes the full matrix directly.
+    """
+
+    def __init__(self, handle, dcodes, doff, qcodes, qoff, matrix, gap_open=10, gap_extend=2, rank=0, world=1,
+                 n_shards=None, pg=None, backend="nccl", alphabet_size=24, rate=None):
+        import torch
+        self.h, self.rank, self.world, self.pg, self.backend = handle, rank, world, pg, backend
+        self.matrix, self.gs, self.ge = matrix, gap_open, gap_extend
+        doff = np.asarray(doff, dtype=np.int64)
+        qoff = np.asarray(qoff, dtype=np.int64)
+        self.Q, self.N = len(qoff) - 1, len(doff) - 1
+        n_shards = n_shards or (4 * world if world > 1 else 1)
+        self.shards = shard_cut(doff, n_shards)
+        lens = np.diff(doff)
+        res = [int(lens[s].sum()) for s in self.shards]
+        self.plan = place(np.diff(qoff), self.shards, res, world, rate=rate)
+        self.blocks = local_blocks(self.plan, rank)
+        dev = torch.device("cuda", handle.device)
+        self.dev = dev
+        self.dbs = {}
+        for s, _qs in self.blocks:
+            self.dbs[s] = handle.load_db(*subset(dcodes, doff, self.shards[s]), alphabet_size=alphabet_size)
+        tabs = assembly_tables(self.plan)
+        self.cap = tabs[3]
+        single = world == 1 and len(self.blocks) == 1 and len(self.blocks[0][1]) == self.Q \
+            and np.array_equal(self.shards[self.blocks[0][0]], np.arange(self.N))
+        self.flat = torch.zeros(self.cap, dtype=torch.int32, device=dev)
+        self.full = None
+        self.asm = None
+        if single:
+            self.full = self.flat[:self.Q * self.N].view(self.Q, self.N)
+        elif rank == 0:
+            self.full = torch.zeros((self.Q, self.N), dtype=torch.int32, device=dev)
+            self.asm = handle.assembly(tabs[0], tabs[1], tabs[2], self.Q, self.N)
+        self.gathered = (torch.empty(world * self.cap, dtype=torch.int32, device=dev) if world > 1
+                         else self.flat)
+        self.jobs = []
+        pos = 0
+        for s, qs in self.blocks:
+            qc, qo = subset(qcodes, qoff, qs)
+            n = len(self.shards[s])
+            self.jobs.append((s, qs, qc, qo, self.flat[pos:pos + len(qs) * n].view(len(qs), n)))
+            pos += len(qs) * n
+
+    def search_local(self, stream=None, host_out=None):
+        for k, (s, _qs, qc, qo, view) in enumerate(self.jobs):
+            out = view if host_out is None else host_out[k]
+            self.h.search(qc, qo, self.dbs[s], self.matrix, self.gs, self.ge, out=out, stream=stream)
+
+    def exchange(self, stream=None):
+        """All-gather of the flat blocks, then rank 0's merge (no-op at N = 1, one shard)."""
+        import torch
+        if self.world > 1:
+            if self.backend == "nccl":
+                self.pg.all_gather_into_tensor(self.gathered, self.flat)
+            else:  # gloo: host staging (functional runs only)
+                torch.cuda.synchronize(self.dev)
+                g = torch.empty(self.world * self.cap, dtype=torch.int32)
+                self.pg.all_gather_into_tensor(g, self.flat.cpu())
+                self.gathered.copy_(g)
+        if self.asm is not None:
+            self.asm(self.gathered, self.full, stream=stream)
+
+    def step(self, stream=None):
+        """One pass of the whole path; returns the device scores[Q][N] on rank 0 (else None)."""
+        self.search_local(stream)
+        self.exchange(stream)
+        return self.full
+
+    def local_cells(self) -> float:
+        return float(sum(float(np.diff(qo).sum()) * float(self.dbs[s].info()["n_residues"])
+                         for s, _q, _qc, qo, _v in self.jobs))
 
 
 def run(plan: Plan, rank: int, n_queries: int, n_seqs: int, score_block, dist=None, device=None,

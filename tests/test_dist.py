@@ -64,7 +64,7 @@ def test_place_covers_every_task():
         assert seen == sorted(plan.tasks)
         loads = np.zeros(g)
         for (q, s), o in zip(plan.tasks, plan.owner):
-            loads[o] += ql[q] * res[s]
+            loads[o] += swdist.gpu_task_time(ql[q], res[s])     # the calibrated model place() uses
         assert loads.max() == pytest.approx(plan.makespan)
         assert plan.makespan <= 2 * plan.lam * (1 + 1e-9)
 
@@ -158,3 +158,45 @@ def test_place_hybrid_dp_variant():
     assert len(d.pe) == len(g.pe) == 12
     assert d.makespan <= (1.5 + 0.25) * d.lam * (1 + 1e-9)
     assert d.makespan <= 2 * g.makespan
+
+
+def _emulate_assemble(tabs, gathered, Q, N):
+    """What sw_assemble computes (include/swdual.h), element by element."""
+    blocks, rows, cols, _cap = tabs
+    out = np.full((Q, N), -1, dtype=np.int32)
+    for src_off, row_off, col_off, nr, nc in blocks:
+        for i in range(nr):
+            for k in range(nc):
+                out[rows[row_off + i], cols[col_off + k]] = gathered[src_off + i * nc + k]
+    return out
+
+
+@pytest.mark.parametrize("world,shards", [(1, 1), (2, 8), (3, 5), (4, 16)])
+def test_assembly_tables_match_assemble(world, shards):
+    """The block tables handed to sw_assemble place every gathered score where
+    dist.assemble (the host merge) does, and cover every (query, sequence)."""
+    c = swgen.make_config("c3", n_db=300, q_lens=[50, 144, 30, 75, 9])
+    ql = np.diff(c["qoff"])
+    sh = swdist.shard_cut(c["doff"], shards)
+    res = [int(np.diff(c["doff"])[s].sum()) for s in sh]
+    plan = swdist.place(ql, sh, res, world)
+    tabs = swdist.assembly_tables(plan)
+    cap = tabs[3]
+    Q, N = len(ql), len(c["doff"]) - 1
+    rng = np.random.default_rng(world * 10 + shards)
+    flats = [rng.integers(0, 1000, size=cap).astype(np.int32) for _ in range(world)]
+    gathered = np.concatenate(flats)
+    ref = swdist.assemble(plan, Q, N, flats)
+    got = _emulate_assemble(tabs, gathered, Q, N)
+    assert (got >= 0).all()
+    np.testing.assert_array_equal(got, ref)
+
+
+def test_task_time_model_orders_by_padded_rows():
+    """Calibrated GPU task times: strip-padded rows x residues
+    / rate + a fixed share; a 144-row query costs as much as a 192-row one."""
+    t = swdist.gpu_task_time
+    assert t(144, 1e6) == t(192, 1e6)
+    assert t(193, 1e6) > t(192, 1e6)
+    assert t(0, 1e6) == 0.0 and t(100, 0) == 0.0
+    assert abs(t(9600, 1e8) - (9600 * 1e8 / swdist.RATE + swdist.T_TASK)) < 1e-12

@@ -443,3 +443,65 @@ def test_mapped_db_writes_into_shared_matrix():
         with pytest.raises(sw.SWError):   # host output is refused for a mapped DB
             h.search(qc, qo, dbs[0], sw.blosum62(), 10, 2, out=np.zeros((3, N), dtype=np.int32))
     np.testing.assert_array_equal(got, oracle_scores(qc, qo, dc, do))
+
+
+def test_mapped_db_resets_its_columns():
+    """A mapped DB writes every one of its columns in every query row: a stale
+    positive value (reused buffer) never survives, not for a long pair split
+    over several CTAs (a > 13k-row query) nor for an empty query's zero row."""
+    import torch
+    sw = _pkg()
+    from paper_conf_icpp_kedad_sidhoummmmt14_b200 import dist
+    rng = np.random.default_rng(77)
+    dl = list(rng.integers(3001, 4500, size=6)) + list(rng.integers(1, 400, size=40)) + [0]
+    dc, do = _seqs(dl, rng)
+    qc, qo = _seqs([13500, 0, 300], rng)
+    N = len(dl)
+    shards = dist.shard_cut(do, 2)
+    with sw.Handle(0) as h:
+        full = torch.full((3, N), 30000, dtype=torch.int32, device="cuda")   # stale, above every true score
+        for idx in shards:
+            db = h.load_db(*dist.subset(dc, do, idx), out_index=idx, out_n=N)
+            h.search(qc, qo, db, sw.blosum62(), 10, 2, out=full)
+        torch.cuda.synchronize()
+        got = full.cpu().numpy()
+    np.testing.assert_array_equal(got, oracle_scores(qc, qo, dc, do))
+
+
+def test_searches_on_two_streams_share_the_handle():
+    """Back-to-back searches of one handle on two streams, no host sync between
+    them (the second waits for the first on the device): both exact."""
+    import torch
+    sw = _pkg()
+    rng = np.random.default_rng(78)
+    dc, do = _seqs(list(rng.integers(1, 600, size=300)), rng)
+    qa, qao = _seqs([700, 150, 3300], rng)
+    qb, qbo = _seqs([90, 2000], rng)
+    s1, s2 = torch.cuda.Stream(), torch.cuda.Stream()
+    with sw.Handle(0) as h:
+        h.set_option("overflow_threshold", 60)      # both searches also run the re-score kernel
+        db = h.load_db(dc, do)
+        oa = torch.empty((3, 300), dtype=torch.int32, device="cuda")
+        ob = torch.empty((2, 300), dtype=torch.int32, device="cuda")
+        for _ in range(3):
+            h.search(qa, qao, db, sw.blosum62(), 10, 2, out=oa, stream=s1)
+            h.search(qb, qbo, db, sw.blosum62(), 10, 2, out=ob, stream=s2)
+        torch.cuda.synchronize()
+        ga, gb = oa.cpu().numpy(), ob.cpu().numpy()
+    np.testing.assert_array_equal(ga, oracle_scores(qa, qao, dc, do))
+    np.testing.assert_array_equal(gb, oracle_scores(qb, qbo, dc, do))
+
+
+def test_overflow_threshold_is_clamped():
+    """A forced threshold above 32767 - S_max is lowered to it, so real int16
+    overflow is still flagged and re-scored exactly."""
+    rng = np.random.default_rng(79)
+    W = 17
+    q = np.full(3300, W, dtype=np.uint8)
+    q[rng.integers(0, 3300, 30)] = rng.integers(0, 20, 30)
+    dc = np.concatenate([q, rng.integers(0, 20, 500).astype(np.uint8)])
+    do = np.array([0, len(q), len(q) + 500], dtype=np.int64)
+    got = gpu_scores(q, np.array([0, len(q)], np.int64), dc, do, opts={"overflow_threshold": 40000})
+    ref = oracle_scores(q, np.array([0, len(q)], np.int64), dc, do)
+    assert ref.max() > 32767
+    np.testing.assert_array_equal(got, ref)

@@ -329,19 +329,27 @@ def run_ours(args):
     # accounting of one step gives its cells and launches (rank-local, then summed)
     h.set_option("timing_accumulate", 0)
     cells_local = 0.0
+    cells_short_local = 0.0
     n_launch_local = 0
     for s_, _qs, qc, qo, view in ss.jobs:
         h.search(qc, qo, ss.dbs[s_], S, 10, 2, out=view, stream=stream)
         one = h.last_stats()
         cells_local += one["cells"]
+        cells_short_local += one["cells_short"]
         n_launch_local += one["n_launches"]
     n_launch_local += 1 if ss.asm is not None else 0
     torch.cuda.synchronize()
-    cells_sum, kms_sum, nl_sum = allreduce([cells_local * args.steps, st["short_ms"], float(n_launch_local)])
+    cells_sum, kms_sum, nl_sum, lms_sum, cshort_sum = allreduce(
+        [cells_local * args.steps, st["short_ms"], float(n_launch_local), st["long_ms"], cells_short_local * args.steps])
     sm_max = clk.get("sm_max_mhz") or 1965.0
     n_sm = torch.cuda.get_device_properties(dev).multi_processor_count
     peak = n_sm * ALU_LANES_PER_SM_CLK * sm_max * 1e6 / OPS_PER_CELL / 1e9
-    achieved = cells_sum / (kms_sum / 1e3) / 1e9 if kms_sum > 0 else None   # per GPU
+    # the dominant kernel: the short-pair (inter-task) kernels, or the long-pair
+    # kernel when it takes longer (C4); its real cells over its CUDA-event time
+    dominant = "short" if kms_sum >= lms_sum else "long"
+    dom_cells = cshort_sum if dominant == "short" else cells_sum - cshort_sum
+    dom_ms = kms_sum if dominant == "short" else lms_sum
+    achieved = dom_cells / (dom_ms / 1e3) / 1e9 if dom_ms > 0 else None   # per GPU
     # algorithmic bytes of one scoring launch: the DB streamed once
     # per query (1 B per residue per query) + the int32 scores written once
     alg_bytes = int(Q * int(d_lens.sum()) + 4 * Q * N) // max(world, 1)
@@ -431,7 +439,9 @@ def run_ours(args):
                              "traffic_unit": "DRAM bytes per launch of the scoring kernel (profiles/traffic.json, ncu)",
                              "algorithmic_bytes_per_launch": alg_bytes,
                              "algorithmic_bytes_basis": "SURVEY 8(d): 1 B per DB residue per query + 4 B per score",
-                             "kernel": "inter_kernel (the persistent scoring launch: long and short pairs), CUDA events around each launch",
+                             "kernel": ("short-pair kernels (short_kernel_q2 / short_kernel_m0)" if dominant == "short"
+                                        else "long-pair kernel (long_kernel)") +
+                                       ": its real cells / its CUDA-event time (events on its launch stream)",
                              "peak_basis": f"{n_sm} SMs x {ALU_LANES_PER_SM_CLK} ALU-pipe lanes/clk x {sm_max:.0f} MHz / "
                                            f"{OPS_PER_CELL} ALU lane-ops per cell (minimal s16x2 Gotoh update; "
                                            f"derived from unit counts + measured pipe attribution)",
@@ -444,6 +454,7 @@ def run_ours(args):
                 "clocks": clk,
                 "detail": {"search_ms_per_step": round(T / args.steps, 3),
                            "scoring_kernel_ms_per_step_per_gpu": round(kms_sum / max(world, 1) / args.steps, 3),
+                           "long_kernel_ms_per_step_per_gpu": round(lms_sum / max(world, 1) / args.steps, 3),
                            "cells_per_step": total_cells, "placement_makespan_model_s": ss.plan.makespan}}
         print(json.dumps(line), flush=True)
     h.close()

@@ -212,11 +212,11 @@ int32_t sw_db_info(sw_db_t db, sw_db_info_t* out);
 
 typedef struct {
   double cells;            /* sum_q m_q * sum_d n_d of the last search (real residues)      */
-  double cells_short;      /* of which in pairs of length <= 3000 (the bulk launches)        */
+  double cells_short;      /* of which scored by the short-pair (inter-task) kernels         */
   double cells_computed;   /* cell updates issued incl. row/column padding and wave fill     */
-  double short_ms;         /* summed CUDA-event time of the scoring launches (the persistent  */
-                           /* kernel covers long AND short pairs of the search)             */
-  double long_ms;          /* reserved (0): long pairs run inside the same persistent launch */
+  double short_ms;         /* summed CUDA-event time of the short-pair kernel launches        */
+  double long_ms;          /* CUDA-event time of the long-pair (intra-task) kernel, which    */
+                           /* runs concurrently with them on the handle's side stream       */
   double search_ms;        /* device time of the whole search, first upload to last kernel   */
   int32_t n_launches;      /* kernels launched by the last search                           */
   int32_t n_score_launches;/* of which scoring (inter-task) kernels                         */
@@ -230,7 +230,8 @@ int32_t sw_last_stats(sw_handle_t h, sw_stats_t* out);
 /*
  * Integer options (testing / tuning).  Keys:
  *   "overflow_threshold"  force the int16 re-score threshold (0 = automatic)
- *   "force_G", "force_R"  force the inter-task lane-group geometry (0 = auto)
+ *   "force_G", "force_R"  force the inter-task lane-group geometry of both short-pair
+ *                         kernels (0 = auto; G in {4, 8, 16, 32}, R in {8, 12, .., 32})
  *   "query_pairs"         1 (default): queries are paired two per s16x2 register for
  *                         the short DB pairs (no PRMT); 0: one query per register
  *   "t_long"              >= 0: DB pairs longer than this are always scored in the
@@ -238,8 +239,6 @@ int32_t sw_last_stats(sw_handle_t h, sw_stats_t* out);
  *                         automatic (pairs whose one-lane-group critical path
  *                         would outlast the search's average share, and every
  *                         pair > 3000 when such pairs hold most of the residues)
- *   "pack_long"           1: pack several long pairs per CTA when a query has
- *                         fewer intra-task strips than warps (default 0)
  *   "bank_copy"           1: shared-memory strip profiles as bank-spread copies
  *                         with 128-byte letter rows (default 1), 0: one copy
  *   "pack_queries"        1: a query-pair slot's shorter half carries further
@@ -247,14 +246,6 @@ int32_t sw_last_stats(sw_handle_t h, sw_stats_t* out);
  *   "bank_skew"           1: single-query profile copies one per lane group of
  *                         a shared-memory phase at searched bank skews
  *                         (conflict-free; default 1), 0: the linear layout
- *   "wide_profile"        1: single-query slots use 32-bit profile rows and
- *                         build each cell pair's scores with one IMAD instead
- *                         of a PRMT (separate kernel; default 0: measured
- *                         neutral)
- *   "resident_strips"     1: a multi-strip query slot whose whole profile fits
- *                         in the CTA's shared-memory share keeps every strip
- *                         resident (no per-pass reload), 0: one strip at a
- *                         time (default 0: measured neutral)
  *   "timing"              1/0, same as SW_FLAG_TIMING
  *   "timing_accumulate"   1: short_ms/long_ms of sw_last_stats sum every search
  *                         since the last "timing_reset" (0: the last search only)

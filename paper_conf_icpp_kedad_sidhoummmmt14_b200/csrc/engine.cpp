@@ -95,11 +95,13 @@ struct sw_handle_s {
   std::vector<sw_db_s*> dbs;
   std::vector<sw_assembly_s*> assemblies;
   // scratch (grown on demand)
-  DevBuf qcodes, qoff, matrix, prof, bbuf, bbuf_long, counters, ovf, ovf_count, scores_tmp, rbuf, qdesc;
-  DevBuf glinks, gflags;  // superstrip boundary rows and their counters (long pairs)
+  DevBuf qcodes, qoff, matrix, prof, bbuf1, bbuf0, wrap, counters, ovf, ovf_count, scores_tmp, rbuf, qdesc;
   DevBuf rgrows, rflags;  // re-score: CTA-to-CTA rows, counters
-  DevBuf imap;            // short work item order
+  DevBuf imap;            // short work item order (mode 1 items, then mode 0 items)
   DevBuf vq, sinfo;       // packed mode-1 slots: strip-padded query codes per half, per-strip info
+  cudaStream_t side = nullptr;             // the long-pair kernel's stream when short pairs run too
+  cudaEvent_t ev_fork = nullptr, ev_join = nullptr;
+
   cudaEvent_t ev_begin = nullptr, ev_end = nullptr;
   // the previous search's completion: a search on another stream waits for it on the
   // device, because both use this handle's scratch
@@ -116,10 +118,6 @@ struct sw_handle_s {
   int64_t opt_pack_queries = 1; // mode-1 slots: fill the shorter half with further queries (strip-aligned)
   int64_t opt_bank_copy = 1;    // query-pair profile: second smem copy shifted by 64 B for odd lane groups
   int64_t opt_bank_skew = 1;    // mode-0 profile copies: per-copy bank skew (mode0_copies)
-  int64_t opt_wide0 = 0;        // single-query slots: 32-bit profile, pair build by IMAD instead of PRMT
-  int64_t opt_resident = 0;     // multi-strip slots whose whole profile fits: all strips resident in smem
-                                // (same-box A/B: neutral within 0.2% on C1-C3, Table V; kept off)
-  int64_t opt_pack_long = 0;    // 1: several long pairs per CTA item when a query has fewer strips than warps
   int64_t opt_align_ws_mb = 2048;  // sw_align: traceback-code workspace per batch
   // sw_align scratch (separate from sw_search's: a search may still be running on another stream)
   DevBuf a_qcodes, a_qoff, a_matrix, a_items, a_links, a_trace, a_best, a_ops, a_out, a_counter;
@@ -143,9 +141,8 @@ struct sw_db_s {
   // per-DB constants of the pair table (computed once at load)
   double sum_short_len = 0, sum_long_len = 0, short_res = 0;
   int32_t max_short = 0, max_long = 0;
-  std::vector<int64_t> lofs_host;   // [np+1] prefix of (len + 72): boundary-row offsets
   std::vector<int64_t> len_prefix;  // [np+1] prefix of padded pair lengths
-  DevBuf dlofs;
+  std::vector<double> res_prefix;   // [np+1] prefix of real residues (both halves)
   DevBuf stream, dpairs;
   std::vector<int64_t> seq_loc;  // caller index -> 2 * pair + half (-1: empty); built on first sw_align
   // output mapping (sw_load_db_mapped): scores of sequence d land in column out_index[d] of
@@ -242,8 +239,8 @@ static ProfGeom make_geom(int G, int R, int m, int alpha, bool long_mode = false
   g.G = G;
   g.R = R;
   g.UB = (R % 8 == 0) ? 8 : 4;
-  g.il = (long_mode && SW_LONG_IL) ? 1 : 0;
-  g.LB = long_mode ? (SW_LONG_IL ? g.UB : R) : ((R % 8 == 0) ? (((R / 8) | 1) * 8) : (((R / 4) | 1) * 4));
+  g.il = long_mode ? 1 : 0;
+  g.LB = long_mode ? g.UB : ((R % 8 == 0) ? (((R / 8) | 1) * 8) : (((R / 4) | 1) * 4));
   g.LS = long_mode ? G * R : G * g.LB;
   if (pad128) g.LS = ((g.LS + 127) / 128) * 128;
   g.NL = alpha + 1;
@@ -278,7 +275,12 @@ static void choose_geom(const sw_handle_s* h, const std::vector<std::pair<int, i
   R = 24;
   for (int g : Gs) {
     for (int r : Rs) {
-      const double per_cell = 1.0 + 7.0 / (5.5 * r) + (r > 24 ? 0.06 : 0.0);
+      // per-step overhead amortised over r rows; a lane of one sub-lane (r % 8 != 0)
+      // has half the ILP.  The single-query kernel spills above 24 rows; the
+      // query-pair kernel (its own register budget) does not lose at 32 (C3 A/B:
+      // (4,32) 7,034 vs (4,24) 6,902 vs (4,20) 6,496 GCUPS, profiles/r02_ab_geometry.txt).
+      const bool qp = !slots.empty() && slots[0].second == 1;
+      const double per_cell = 1.0 + 7.0 / (5.5 * r) + (r % 8 ? 0.06 : 0.0) + (!qp && r > 24 ? 0.06 : 0.0);
       double cost = 0;
       for (auto [m, mode] : slots) {
         const int strips = std::max(1, (m + g * r - 1) / (g * r));
@@ -347,18 +349,12 @@ int32_t sw_set_option(sw_handle_t h, const char* key, int64_t value) {
   } else if (k == "align_workspace_mb") {
     if (value < 1) return set_err(h, SW_EINVAL, "sw_set_option: align_workspace_mb must be >= 1");
     h->opt_align_ws_mb = value;
-  } else if (k == "pack_long") {
-    h->opt_pack_long = value;
   } else if (k == "pack_queries") {
     h->opt_pack_queries = value;
   } else if (k == "bank_copy") {
     h->opt_bank_copy = value;
   } else if (k == "bank_skew") {
     h->opt_bank_skew = value;
-  } else if (k == "wide_profile") {
-    h->opt_wide0 = value;
-  } else if (k == "resident_strips") {
-    h->opt_resident = value;
   } else if (k == "query_pairs") {
     h->opt_query_pairs = value;
   } else if (k == "timing_accumulate") {
@@ -415,16 +411,15 @@ int32_t sw_load_db(sw_handle_t h, const uint8_t* codes, const int64_t* offsets, 
       }
     }
     std::vector<uint16_t>& stream = P.stream;
-    {  // boundary-row offsets of every pair (any pair may be a long item for a tall query)
-      db->lofs_host.assign(np + 1, 0);
+    {  // prefix sums over the pairs (longest first): padded columns, real residues
       db->len_prefix.assign(np + 1, 0);
+      db->res_prefix.assign(np + 1, 0.0);
       for (size_t p = 0; p < np; ++p) {
-        db->lofs_host[p + 1] = db->lofs_host[p] + db->pairs[p].len + 72;
-        db->len_prefix[p + 1] = db->len_prefix[p] + db->pairs[p].len;
+        const PairRec& r = db->pairs[p];
+        db->len_prefix[p + 1] = db->len_prefix[p] + r.len;
+        db->res_prefix[p + 1] = db->res_prefix[p] + double(db->seq_len[size_t(r.id0)]) +
+                                (r.id1 >= 0 ? double(db->seq_len[size_t(r.id1)]) : 0.0);
       }
-      SW_CK(db->dlofs.ensure(db->lofs_host.size() * sizeof(int64_t)));
-      SW_CK(cudaMemcpyAsync(db->dlofs.p, db->lofs_host.data(), db->lofs_host.size() * sizeof(int64_t),
-                            cudaMemcpyHostToDevice, st));
     }
     SW_CK(db->stream.ensure(stream.size() * sizeof(uint16_t)));
     SW_CK(db->dpairs.ensure(std::max<size_t>(np, 1) * sizeof(PairRec)));
@@ -510,8 +505,9 @@ static std::pair<cudaEvent_t, cudaEvent_t>* next_event_pair(sw_handle_s* h) {
   return &h->events[h->n_events_used++];
 }
 
-// The scoring launch: profiles of every query, then ONE persistent kernel over
-// all (query, long pair) and (query, short chunk) work items.
+// The scoring launches of one search: profiles of every query, then the
+// long-pair (intra-task) kernel (concurrently, when short pairs are scored too)
+// and one persistent short-pair kernel per mode present (query pairs, single query).
 struct LaunchCtx {
   sw_handle_s* h;
   sw_db_s* db;
@@ -523,12 +519,23 @@ struct LaunchCtx {
   int64_t ovf_cap;
   uint32_t nGe, nGsGe;
   bool timing;
-  double sum_short;      // sum of short pair lengths
-  int32_t max_short, max_long;
 };
 
+struct LaunchOut {
+  double cells_computed = 0, cells_short = 0;
+  int launches = 0;
+};
+
+static void record_begin(sw_handle_s* h, bool timing, int kind, cudaStream_t st, std::pair<cudaEvent_t, cudaEvent_t>*& ev) {
+  ev = timing ? next_event_pair(h) : nullptr;
+  if (ev) {
+    h->event_kind[h->n_events_used - 1] = kind;
+    SW_CK(cudaEventRecord(ev->first, st));
+  }
+}
+
 static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std::vector<int64_t>& qoff0,
-                       double& cells_computed, int& launches) {
+                       LaunchOut& out) {
   sw_handle_s* h = c.h;
   sw_db_s* db = c.db;
   const int alpha = db->alpha;
@@ -540,57 +547,44 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
   std::stable_sort(order.begin(), order.end(), [&](int x, int y) { return qlen[size_t(x)] > qlen[size_t(y)]; });
   std::vector<int> ms;
   for (int i : order) ms.push_back(int(qlen[size_t(i)]));
-  // geometry from the plain neighbour pairing (mode 1: two queries per register)
   const bool pairs_on = h->opt_query_pairs != 0;
-  std::vector<std::pair<int, int>> slot_m;
+  // geometry per mode from the plain neighbour pairing (mode 1: two queries per register)
+  std::vector<std::pair<int, int>> m1, m0;
   for (size_t k = 0; k < order.size();) {
-    if (pairs_on && k + 1 < order.size()) { slot_m.push_back({ms[k], 1}); k += 2; }
-    else { slot_m.push_back({ms[k], 0}); k += 1; }
+    if (pairs_on && k + 1 < order.size()) { m1.push_back({ms[k], 1}); k += 2; }
+    else { m0.push_back({ms[k], 0}); k += 1; }
   }
   const int nshort_db = np - db->n_long;  // (only for the geometry cost model)
-  int G = 4, R = 24;
+  const double Lavg = nshort_db > 0 ? db->sum_short_len / nshort_db : 1.0;
   double qsum = 0;
   for (int m : ms) qsum += m;
-  choose_geom(h, slot_m, nshort_db > 0 ? db->sum_short_len / nshort_db : 1.0, G, R, double(db->max_short),
-              qsum * double(db->n_res));
-  if (!inter_config_supported(G, R)) fail(SW_EUNSUPPORTED, "no kernel for this geometry");
-  const int NT = inter_block_threads(), NG = NT / G, W = NT / 32;
-  const int LB2 = (((R / 4) | 1) * 16);
-  // Query-pair profile rows are LDS.128 per lane: a quarter-warp phase holds two
-  // G = 4 groups reading random letters.  With LS2 a multiple of 128 B and odd
-  // groups reading a second copy shifted by 64 B, the two groups always hit
-  // disjoint bank halves ({k*LB2} mod 128 and {k*LB2 + 64} mod 128 partition
-  // the eight 16-byte slots when LB2 is an odd multiple of 16).
-  const bool bank_copy = h->opt_bank_copy != 0;
-  const int LS2 = bank_copy ? ((G * LB2 + 127) / 128) * 128 : G * LB2;
-  const int SB2 = (((alpha + 1) * LS2 + 15) / 16) * 16;
-  // copies: lanes of one phase (128 B / unit) divided by the group width
-  const int ncopy2 = bank_copy ? std::max(1, (128 / 16) / G) : 1;
-  // Per slot, pairs [0, nlong) go to the intra-task (long) mode: a short item
-  // (one lane group, every strip of its query in turn) must not run much longer
-  // than an average lane group's share of the whole launch, or it becomes the
-  // tail.  Optional override: "t_long" forces every pair longer than it there.
+  int G1 = 4, R1 = 24, G0 = 4, R0 = 24;
+  if (!m1.empty()) choose_geom(h, m1, Lavg, G1, R1, double(db->max_short), qsum * double(db->n_res));
+  if (!m0.empty()) choose_geom(h, m0, Lavg, G0, R0, double(db->max_short), qsum * double(db->n_res));
+  if (!m1.empty() && !short_config_supported(1, G1, R1)) fail(SW_EUNSUPPORTED, "no query-pair kernel for this geometry");
+  if (!m0.empty() && !short_config_supported(0, G0, R0)) fail(SW_EUNSUPPORTED, "no single-query kernel for this geometry");
+  const int NT = SCORE_NT, NG1 = NT / G1, NG0 = NT / G0, W = LONG_W;
   auto pairs_longer_than = [&](int64_t Lc) {  // pairs are sorted longest first
     int lo = 0, hi = np;
     while (lo < hi) { const int mid = (lo + hi) / 2; if (db->pairs[size_t(mid)].len > Lc) lo = mid + 1; else hi = mid; }
     return lo;
   };
-  // Short-pair slots.  Mode 1: half A (low) and half B (high) each hold a list
-  // of queries laid end to end on strip boundaries; the slot runs max(strips A,
-  // strips B) strips.  The longest unplaced query opens a slot as half A and
-  // half B takes the subset of the remaining queries whose strips best fill it
-  // (subset sum), so the shorter half carries further queries instead of PAD
-  // rows.  A last odd query runs alone in mode 0 (two DB sequences per register).
+  // Short-pair slots.  Mode 1: half A (low) and half B (high) each hold a list of
+  // queries laid end to end on strip boundaries; the slot runs max(strips A,
+  // strips B) strips.  The longest unplaced query opens a slot as half A and half
+  // B takes the subset of the remaining queries whose strips best fill it (subset
+  // sum), so the shorter half carries further queries instead of PAD rows.  A
+  // last odd query runs alone in mode 0 (two DB sequences per register).
   struct Slot { int mode; std::vector<int> A, B; int strips, nlong; };
   std::vector<Slot> slots;
   {
-    auto nst = [&](int k) { return std::max(1, (ms[size_t(k)] + G * R - 1) / (G * R)); };
+    auto nst1 = [&](int k) { return std::max(1, (ms[size_t(k)] + G1 * R1 - 1) / (G1 * R1)); };
     std::vector<int> rem;
     for (size_t k = 0; k < order.size(); ++k) rem.push_back(int(k));  // longest first
     while (pairs_on && rem.size() >= 2) {
       const int a0 = rem[0];
       rem.erase(rem.begin());
-      const int target = nst(a0);
+      const int target = nst1(a0);
       std::vector<int> B;
       if (h->opt_pack_queries && double(rem.size()) * target <= 4e6) {
         // best subset sum <= target over rem (0/1 knapsack on strip counts)
@@ -599,14 +593,14 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
         std::vector<int> bestv(size_t(target) + 1, -1);
         bestv[0] = 0;
         for (size_t i = 0; i < n; ++i) {
-          const int w = nst(rem[i]);
+          const int w = nst1(rem[i]);
           for (int v = target; v >= w; --v)
             if (bestv[size_t(v - w)] >= 0 && bestv[size_t(v)] < 0) { bestv[size_t(v)] = 1; take[i][size_t(v)] = 1; }
         }
         int v = target;
         while (v > 0 && bestv[size_t(v)] < 0) --v;
         for (size_t i = n; i-- > 0 && v > 0;)
-          if (take[i][size_t(v)]) { B.push_back(rem[i]); v -= nst(rem[i]); }
+          if (take[i][size_t(v)]) { B.push_back(rem[i]); v -= nst1(rem[i]); }
       } else {
         B.push_back(rem[0]);  // plain neighbour pairing
       }
@@ -614,20 +608,23 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
       for (int b : B) rem.erase(std::find(rem.begin(), rem.end(), b));
       slots.push_back({1, {a0}, B, target, 0});
     }
-    for (int k : rem) slots.push_back({0, {k}, {}, nst(k), 0});
+    for (int k : rem) slots.push_back({0, {k}, {}, std::max(1, (ms[size_t(k)] + G0 * R0 - 1) / (G0 * R0)), 0});
   }
-  const int VG = G * (R % 8 == 0 ? 2 : 1);
-  double group_steps = 0;  // wavefront steps of all short work if nothing went long
+  // Long pairs per slot: a short item (one lane group, every strip of its slot in
+  // turn) must not run much longer than an average lane group's share of the
+  // whole search, or it becomes the tail.  Pairs [0, nlong) of a slot go to the
+  // intra-task kernel.  Option "t_long" forces every pair longer than it there.
+  double group_steps = 0, resident_groups = 0;  // wavefront steps of all short work if nothing went long
   for (auto& sl : slots) {
-    const int strips = sl.strips;
+    const int VG = sl.mode == 1 ? G1 * (R1 % 8 == 0 ? 2 : 1) : G0 * (R0 % 8 == 0 ? 2 : 1);
     const double seqs = sl.mode == 1 ? 2.0 * np : double(np);
     const double cols = sl.mode == 1 ? 2.0 * db->len_prefix[size_t(np)] : double(db->len_prefix[size_t(np)]);
-    group_steps += double(strips) * (cols + seqs * VG);
+    group_steps += double(sl.strips) * (cols + seqs * VG);
   }
-  const double resident_groups = 2.0 * h->sms * NG;
+  resident_groups = 2.0 * h->sms * double(!m1.empty() ? NG1 : NG0);
   const double crit = std::max(double(CRIT_MIN_STEPS), CRIT_FRACTION * group_steps / resident_groups);
   // Long-sequence databases (most residues in pairs longer than T_LONG, config 4)
-  // are scored entirely by the intra-task mode; otherwise the critical-path
+  // are scored entirely by the intra-task kernel; otherwise the critical-path
   // rule alone decides.
   int nlong_opt = 0;
   if (h->opt_t_long >= 0) {
@@ -636,19 +633,24 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
     const int nT = pairs_longer_than(T_LONG);
     if (double(db->len_prefix[size_t(nT)]) > 0.5 * double(db->len_prefix[size_t(np)])) nlong_opt = nT;
   }
-  int nlong_max = 0;
-  for (auto& sl : slots) {
-    const int strips = sl.strips;
-    const int64_t Lc = int64_t(crit / strips);
-    sl.nlong = std::max(nlong_opt, pairs_longer_than(Lc));
-    nlong_max = std::max(nlong_max, sl.nlong);
-  }
+  for (auto& sl : slots) sl.nlong = std::max(nlong_opt, pairs_longer_than(int64_t(crit / sl.strips)));
   std::vector<int> qnlong(order.size(), 0);
   for (auto& sl : slots) {
     for (int k : sl.A) qnlong[size_t(k)] = sl.nlong;
     for (int k : sl.B) qnlong[size_t(k)] = sl.nlong;
   }
-  // profiles: long geometry per query; short geometry per slot
+  // ---- profiles: long geometry per query (if it has long pairs); short geometry per slot
+  const int LB2 = (((R1 / 4) | 1) * 16);
+  // Query-pair profile rows are LDS.128 per lane: a quarter-warp phase holds two
+  // G = 4 groups reading random letters.  With LS2 a multiple of 128 B and odd
+  // groups reading a second copy shifted by 64 B, the two groups always hit
+  // disjoint bank halves ({k*LB2} mod 128 and {k*LB2 + 64} mod 128 partition the
+  // eight 16-byte slots when LB2 is an odd multiple of 16).
+  const bool bank_copy = h->opt_bank_copy != 0;
+  const int LS2 = bank_copy ? ((G1 * LB2 + 127) / 128) * 128 : G1 * LB2;
+  const int SB2 = (((alpha + 1) * LS2 + 15) / 16) * 16;
+  const int ncopy2 = bank_copy ? std::max(1, (128 / 16) / G1) : 1;
+  const ProfGeom g0 = make_geom(G0, R0, 1, alpha, false, bank_copy);  // SB / LS / LB of the mode-0 profile
   size_t total = 0;
   std::vector<ProfGeom> gl;
   std::vector<size_t> off_l;
@@ -657,15 +659,10 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
     off_l.push_back(total);
     total += qnlong[k] > 0 ? size_t(gl.back().n_strips) * gl.back().SB : 0;
   }
-  const ProfGeom g1 = make_geom(G, R, 1, alpha, false, bank_copy);  // SB / LS / LB of the mode-0 profile
-  const bool wide0 = h->opt_wide0 != 0 && inter_wide_supported(G, R);  // mode-0 slots use the 32-bit profile (two sub-lanes only)
   std::vector<size_t> off_s;
-  std::vector<int> strips_s;
   for (auto& sl : slots) {
-    const int n = sl.strips;
-    strips_s.push_back(n);
     off_s.push_back(total);
-    if (sl.nlong < np) total += size_t(n) * ((sl.mode == 1 || wide0) ? SB2 : g1.SB);
+    if (sl.nlong < np) total += size_t(sl.strips) * (sl.mode == 1 ? SB2 : g0.SB);
   }
   SW_CK(h->prof.ensure(total + 16));
   uint8_t* prof = h->prof.as<uint8_t>();
@@ -674,52 +671,42 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
   auto pair_len_sum = [&](int p0, int p1) {  // sum of padded pair lengths over [p0, p1)
     return double(db->len_prefix[size_t(p1)] - db->len_prefix[size_t(p0)]);
   };
-  std::vector<QueryDesc> desc(order.size());
-  int64_t long_items = 0, flags_total = 0, glink_total = 0, done_total = 0;
-  int max_lstrips = 1;
-  for (size_t k = 0; k < order.size(); ++k) {
-    const int qi = order[k];
-    const int nl = qnlong[k];
-    if (nl > 0) {
-      SW_CK(launch_build_profile(qptr(int(k)), ms[k], dmat, alpha, gl[k], prof + off_l[k], c.st));
-      ++launches;
-      max_lstrips = std::max(max_lstrips, gl[k].n_strips);
-    }
-    QueryDesc& d = desc[k];
-    d.prof = nullptr;
-    d.prof_long = prof + off_l[k];
-    d.scores = c.dscores + int64_t(qi) * db->out_n;
-    d.n_strips = 0;
-    d.n_strips_long = gl[k].n_strips;
-    d.qidx = qi;
-    d.n_long = nl;
-    // CTAs per long pair: enough to split very tall queries, few enough that each
-    // CTA still runs ~LONG_ROUNDS rounds of W strips (amortises the pipeline ramp)
-    d.n_super = std::max(1, (gl[k].n_strips + W * LONG_ROUNDS - 1) / (W * LONG_ROUNDS));
-    // a query with fewer strips than warps: several pairs per CTA item
-    d.pairs_per_item = (h->opt_pack_long && gl[k].n_strips < W) ? W / gl[k].n_strips : 1;
-    if (d.pairs_per_item > 1) d.n_super = 1;
-    d.pad2_ = 0;
-    d.long_item_begin = int(long_items);
-    d.flag_base = int(flags_total);
-    d.done_base = int(done_total);
-    d.glink_base = glink_total;
-    d.glink_stride = db->lofs_host[size_t(nl)];
-    const int64_t items_q = d.pairs_per_item > 1 ? (nl + d.pairs_per_item - 1) / d.pairs_per_item
-                                                  : int64_t(nl) * d.n_super;
-    long_items += items_q;
-    flags_total += int64_t(nl) * d.n_super;
-    done_total += nl;
-    if (d.n_super > 1) glink_total += int64_t(d.n_super) * d.glink_stride;
-    cells_computed += 2.0 * (pair_len_sum(0, nl) + 32.0 * nl) * double(gl[k].n_strips) * 32 * LONG_R;
+  auto pair_res_sum = [&](int p0, int p1) { return db->res_prefix[size_t(p1)] - db->res_prefix[size_t(p0)]; };
+  // single-query searches with long pairs run as ONE combined launch (long items
+  // first, one pair per item); otherwise the long kernel packs short queries' pairs
+  bool any_q2 = false, any_m0 = false, any_long = false;
+  for (auto& sl : slots) {
+    if (sl.nlong < np) (sl.mode == 1 ? any_q2 : any_m0) = true;
+    if (sl.nlong > 0) any_long = true;
   }
+  const bool combined = any_long && any_m0 && !any_q2;
+  // ---- long work: one item per (query, long pair), or per `pack` pairs
+  std::vector<LongQuery> ldesc;
+  int64_t long_items = 0;
+  int32_t max_long = 0;
+  for (size_t k = 0; k < order.size(); ++k) {
+    const int nl = qnlong[k];
+    if (nl <= 0) continue;
+    SW_CK(launch_build_profile(qptr(int(k)), ms[k], dmat, alpha, gl[k], prof + off_l[k], c.st));
+    ++out.launches;
+    LongQuery d{};
+    d.prof_long = prof + off_l[k];
+    d.scores = c.dscores + int64_t(order[k]) * db->out_n;
+    d.n_strips = gl[k].n_strips;
+    d.qidx = order[k];
+    d.item_begin = int(long_items);
+    d.n_long = nl;
+    d.pack = (combined || gl[k].n_strips >= W) ? 1 : W / gl[k].n_strips;
+    ldesc.push_back(d);
+    long_items += (nl + d.pack - 1) / d.pack;
+    max_long = std::max(max_long, db->pairs[0].len);
+    out.cells_computed += 2.0 * (pair_len_sum(0, nl) + 64.0 * nl) * double(gl[k].n_strips) * 32 * LONG_R;
+  }
+  // ---- short work: slots per mode
   std::vector<SlotDesc> sdesc(slots.size());
-  int item = 0;
-  int min_pb = np;
-  // packed halves: strip-padded code arrays (PAD = alpha) and per-strip info
   size_t vq_total = 0, si_total = 0;
   for (auto& sl : slots)
-    if (sl.mode == 1) { vq_total += 2 * size_t(sl.strips) * G * R; si_total += size_t(sl.strips); }
+    if (sl.mode == 1) { vq_total += 2 * size_t(sl.strips) * G1 * R1; si_total += size_t(sl.strips); }
   std::vector<StripInfo> sinfo(si_total);
   if (vq_total) {
     SW_CK(h->vq.ensure(vq_total));
@@ -727,26 +714,27 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
     SW_CK(h->sinfo.ensure(si_total * sizeof(StripInfo)));
   }
   size_t vq_off = 0, si_off = 0;
+  int min_pb1 = np, min_pb0 = np, max_strips1 = 1, max_strips0 = 1;
   for (size_t j = 0; j < slots.size(); ++j) {
     const Slot& sl = slots[j];
     SlotDesc& d = sdesc[j];
     const int ns = np - sl.nlong;  // short pairs of this slot
+    const int NGm = sl.mode == 1 ? NG1 : NG0;
     d.prof = prof + off_s[j];
     d.mode = sl.mode;
-    d.n_strips = strips_s[j];
+    d.n_strips = sl.strips;
     d.qidx0 = order[size_t(sl.A[0])];
     d.scores0 = c.dscores + int64_t(d.qidx0) * db->out_n;
-    d.qidx1 = -1;
-    d.scores1 = nullptr;
     d.sinfo = nullptr;
-    d.res_stride = 0;
-    d.wide = (sl.mode == 0 && wide0) ? 1 : 0;
-    uint8_t* vA = nullptr;
-    uint8_t* vB = nullptr;
+    d.pair_begin = sl.nlong;
+    d.n_items = ns > 0 ? (sl.mode == 1 ? (2 * ns + NGm - 1) / NGm : (ns + NGm - 1) / NGm) : 0;
+    double rows_real = 0;
+    for (int kq : sl.A) rows_real += ms[size_t(kq)];
+    for (int kq : sl.B) rows_real += ms[size_t(kq)];
     if (sl.mode == 1) {
-      const size_t GR = size_t(G) * R;
-      vA = h->vq.as<uint8_t>() + vq_off;
-      vB = vA + size_t(sl.strips) * GR;
+      const size_t GR = size_t(G1) * R1;
+      uint8_t* vA = h->vq.as<uint8_t>() + vq_off;
+      uint8_t* vB = vA + size_t(sl.strips) * GR;
       vq_off += 2 * size_t(sl.strips) * GR;
       StripInfo* si = sinfo.data() + si_off;
       d.sinfo = h->sinfo.as<StripInfo>() + si_off;
@@ -757,7 +745,7 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
         uint8_t* dst = hf == 0 ? vA : vB;
         int st0 = 0;
         for (int kq : L) {
-          const int n = std::max(1, (ms[size_t(kq)] + G * R - 1) / (G * R));
+          const int n = std::max(1, (ms[size_t(kq)] + G1 * R1 - 1) / (G1 * R1));
           if (ms[size_t(kq)] > 0)
             SW_CK(cudaMemcpyAsync(dst + size_t(st0) * GR, qptr(kq), size_t(ms[size_t(kq)]), cudaMemcpyDeviceToDevice,
                                   c.st));
@@ -766,48 +754,46 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
           st0 += n;
         }
       }
-    }
-    d.pair_begin = sl.nlong;
-    d.item_begin = item;
-    d.n_items = ns > 0 ? (sl.mode == 1 ? (2 * ns + NG - 1) / NG : (ns + NG - 1) / NG) : 0;
-    item += d.n_items;
-    if (ns > 0) {
-      min_pb = std::min(min_pb, sl.nlong);
-      const double sumS = pair_len_sum(sl.nlong, np) + double(ns) * 2 * G;
-      if (sl.mode == 1) {
-        const int rows = sl.strips * G * R;
-        SW_CK(launch_build_profile_q2(vA, rows, vB, rows, dmat, alpha, G, R, LB2, LS2, d.n_strips, SB2,
+      if (ns > 0) {
+        const int rows = sl.strips * G1 * R1;
+        SW_CK(launch_build_profile_q2(vA, rows, vB, rows, dmat, alpha, G1, R1, LB2, LS2, d.n_strips, SB2,
                                       prof + off_s[j], c.st));
-        cells_computed += 2.0 * (2.0 * sumS) * double(d.n_strips) * G * R;  // every sequence, 2 queries
-      } else if (d.wide) {  // low half S[q_i][a], high half 0 (mb < 0)
-        SW_CK(launch_build_profile_q2(qptr(sl.A[0]), ms[size_t(sl.A[0])], nullptr, -1, dmat, alpha, G, R, LB2, LS2,
-                                      d.n_strips, SB2, prof + off_s[j], c.st));
-        cells_computed += 2.0 * sumS * double(d.n_strips) * G * R;
-      } else {
-        ProfGeom gq = g1;
-        gq.n_strips = d.n_strips;
-        SW_CK(launch_build_profile(qptr(sl.A[0]), ms[size_t(sl.A[0])], dmat, alpha, gq, prof + off_s[j], c.st));
-        cells_computed += 2.0 * sumS * double(d.n_strips) * G * R;
+        ++out.launches;
+        const double sumS = pair_len_sum(sl.nlong, np) + double(ns) * 2 * G1;
+        out.cells_computed += 2.0 * (2.0 * sumS) * double(d.n_strips) * G1 * R1;  // every sequence, 2 queries
+        min_pb1 = std::min(min_pb1, sl.nlong);
+        max_strips1 = std::max(max_strips1, sl.strips);
       }
-      ++launches;
+    } else if (ns > 0) {
+      ProfGeom gq = g0;
+      gq.n_strips = d.n_strips;
+      SW_CK(launch_build_profile(qptr(sl.A[0]), ms[size_t(sl.A[0])], dmat, alpha, gq, prof + off_s[j], c.st));
+      ++out.launches;
+      const double sumS = pair_len_sum(sl.nlong, np) + double(ns) * 2 * G0;
+      out.cells_computed += 2.0 * sumS * double(d.n_strips) * G0 * R0;
+      min_pb0 = std::min(min_pb0, sl.nlong);
+      max_strips0 = std::max(max_strips0, sl.strips);
     }
+    if (ns > 0) out.cells_short += rows_real * pair_res_sum(sl.nlong, np);
   }
-  // global order of the short items: k-way merge of the slots' chunk lists
-  // (each already longest-first) by critical path = strips x first pair length
+  // global order of the short items of each mode: k-way merge of the slots' chunk
+  // lists (each already longest-first) by critical path = strips x first pair length
   std::vector<int2> imap;
-  imap.reserve(size_t(item));
-  {
+  int n_items1 = 0, n_items0 = 0;
+  for (int mode = 1; mode >= 0; --mode) {
     struct Head { double key; int slot, chunk; };
     auto cmp = [](const Head& x, const Head& y) { return x.key < y.key || (x.key == y.key && x.slot > y.slot); };
     std::vector<Head> heap;
+    const int NGm = mode == 1 ? NG1 : NG0;
     auto key_of = [&](int j, int ch) {
       const SlotDesc& d = sdesc[size_t(j)];
-      const int p = d.pair_begin + (d.mode == 1 ? (ch * NG) / 2 : ch * NG);
+      const int p = d.pair_begin + (d.mode == 1 ? (ch * NGm) / 2 : ch * NGm);
       return double(d.n_strips) * double(db->pairs[size_t(std::min(p, np - 1))].len + 8);
     };
     for (size_t j = 0; j < sdesc.size(); ++j)
-      if (sdesc[j].n_items > 0) heap.push_back({key_of(int(j), 0), int(j), 0});
+      if (sdesc[j].mode == mode && sdesc[j].n_items > 0) heap.push_back({key_of(int(j), 0), int(j), 0});
     std::make_heap(heap.begin(), heap.end(), cmp);
+    const size_t before = imap.size();
     while (!heap.empty()) {
       std::pop_heap(heap.begin(), heap.end(), cmp);
       Head hd = heap.back();
@@ -818,131 +804,149 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
         std::push_heap(heap.begin(), heap.end(), cmp);
       }
     }
+    (mode == 1 ? n_items1 : n_items0) = int(imap.size() - before);
   }
+  if (long_items + int64_t(imap.size()) >= (int64_t(1) << 31)) fail(SW_EUNSUPPORTED, "too many work items");
   if (si_total)
     SW_CK(cudaMemcpyAsync(h->sinfo.p, sinfo.data(), si_total * sizeof(StripInfo), cudaMemcpyHostToDevice, c.st));
   SW_CK(h->imap.ensure(std::max<size_t>(imap.size(), 1) * sizeof(int2)));
   if (!imap.empty())
     SW_CK(cudaMemcpyAsync(h->imap.p, imap.data(), imap.size() * sizeof(int2), cudaMemcpyHostToDevice, c.st));
-  int max_strips = 1;
-  for (int n : strips_s) max_strips = std::max(max_strips, n);
-  const ProfGeom l0 = gl[0];
-  // copy c of a strip sits at c * cstride; cstride = SB + 128 / ncopy (SB is a
-  // multiple of 128 when copies are used)
-  const Mode0Copies mc0 = mode0_copies(G, R, g1.LB, g1.SB, bank_copy, h->opt_bank_skew != 0);
-  const int ncopy0 = mc0.ncopy, cstride0 = mc0.cstride;
-  const int cstride2 = SB2 + (ncopy2 > 1 ? 128 / ncopy2 : 0);
-  const int sprof_bytes = std::max(mc0.bytes, (ncopy2 - 1) * cstride2 + SB2);
-  // an item is either short or long: the long-mode slots reuse the same bytes
-  int smem = SW_SMEM_UNION ? std::max(sprof_bytes, nlong_max > 0 ? W * l0.SB : 0)
-                                 : sprof_bytes + 128 + (nlong_max > 0 ? W * l0.SB : 0);
-  int occ = inter_max_ctas_per_sm(G, R, NT, smem, wide0);
-  if (occ <= 0) fail(SW_ECUDA, "inter kernel does not fit on an SM");
-  // Resident strips: a multi-strip slot whose strips (with their bank copies) all
-  // fit in the per-CTA shared-memory share of the current occupancy keeps them
-  // resident, so its items load the profile once instead of once per strip pass
-  // (two CTA barriers per pass saved).  Kept only if the occupancy does not drop.
-  if (h->opt_resident) {
-    const int long_part = nlong_max > 0 ? W * l0.SB : 0;
-    const int stride0 = (mc0.bytes + 127) / 128 * 128;
-    const int stride2 = (((ncopy2 - 1) * cstride2 + SB2) + 127) / 128 * 128;
-    const int cap = 233472 / occ - 2048 - (SW_SMEM_UNION ? 0 : long_part);
-    int res_bytes = sprof_bytes;
-    bool any = false;
-    for (size_t j2 = 0; j2 < sdesc.size(); ++j2) {
-      SlotDesc& d = sdesc[j2];
-      const int stride = (d.mode == 1 || d.wide) ? stride2 : stride0;
-      const int64_t need = int64_t(d.n_strips) * stride;
-      if (d.n_items > 0 && d.n_strips > 1 && need <= cap) {
-        d.res_stride = stride;
-        res_bytes = std::max(res_bytes, int(need));
-        any = true;
-      }
-    }
-    if (any) {
-      const int smem_r = SW_SMEM_UNION ? std::max(res_bytes, long_part) : res_bytes + long_part;
-      if (inter_max_ctas_per_sm(G, R, NT, smem_r, wide0) >= occ) {
-        smem = smem_r;
-      } else {
-        for (auto& d : sdesc) d.res_stride = 0;
-      }
-    }
-  }
-  SW_CK(h->qdesc.ensure(desc.size() * sizeof(QueryDesc) + sdesc.size() * sizeof(SlotDesc) + 16));
-  QueryDesc* d_desc = h->qdesc.as<QueryDesc>();
-  SlotDesc* d_slots = reinterpret_cast<SlotDesc*>(d_desc + desc.size());
-  SW_CK(cudaMemcpyAsync(d_desc, desc.data(), desc.size() * sizeof(QueryDesc), cudaMemcpyHostToDevice, c.st));
+  SW_CK(h->qdesc.ensure(ldesc.size() * sizeof(LongQuery) + sdesc.size() * sizeof(SlotDesc) + 16));
+  LongQuery* d_ldesc = h->qdesc.as<LongQuery>();
+  SlotDesc* d_slots = reinterpret_cast<SlotDesc*>(h->qdesc.as<uint8_t>() + ldesc.size() * sizeof(LongQuery));
+  if (!ldesc.empty())
+    SW_CK(cudaMemcpyAsync(d_ldesc, ldesc.data(), ldesc.size() * sizeof(LongQuery), cudaMemcpyHostToDevice, c.st));
   SW_CK(cudaMemcpyAsync(d_slots, sdesc.data(), sdesc.size() * sizeof(SlotDesc), cudaMemcpyHostToDevice, c.st));
-  const int64_t n_items = long_items + item;
-  if (n_items >= (int64_t(1) << 31)) fail(SW_EUNSUPPORTED, "too many work items");
-  const int grid = int(std::max<int64_t>(1, std::min<int64_t>(n_items, int64_t(occ) * h->sms)));
-  const int32_t max_short = min_pb < np ? db->pairs[size_t(min_pb)].len : 0;
-  const int32_t max_long = db->pairs[0].len;
-  const int bcap = ((max_short + 4 * G + 8 + 4) + 3) / 4 * 4;  // wave width up to V*G sub-lanes (V <= 3) + align pad
-  if (max_strips > 1 && min_pb < np) SW_CK(h->bbuf.ensure(size_t(grid) * NG * bcap * sizeof(uint2)));
-  const int lcap = max_long + 64 + 8;
-  if (nlong_max > 0 && max_lstrips > 1) SW_CK(h->bbuf_long.ensure(size_t(grid) * W * lcap * sizeof(uint2)));
-  SW_CK(h->counters.ensure(sizeof(int)));
-  SW_CK(cudaMemsetAsync(h->counters.p, 0, sizeof(int), c.st));
-  const size_t nflags = size_t(std::max<int64_t>(flags_total, 1)), ndone = size_t(std::max<int64_t>(done_total, 1));
-  SW_CK(h->gflags.ensure((nflags + ndone) * sizeof(int)));
-  SW_CK(cudaMemsetAsync(h->gflags.p, 0, (nflags + ndone) * sizeof(int), c.st));
-  if (glink_total > 0) SW_CK(h->glinks.ensure(size_t(glink_total) * sizeof(uint2)));
-  InterArgs a{};
-  a.queries = d_desc;
-  a.n_queries = int(order.size());
-  a.slots = d_slots;
-  a.n_slots = int(slots.size());
-  a.n_short_items = item;
-  a.item_map = h->imap.as<int2>();
-  a.SB2 = SB2;
-  a.ncopy[0] = ncopy0;
-  a.ncopy[1] = ncopy2;
-  a.cstride[0] = cstride0;
-  a.cstride[1] = cstride2;
-  a.cskew0 = mc0.skew;
-  a.wmul = 65536u;
-  a.LS2 = LS2;
-  a.LB2 = LB2;
-  a.SB = g1.SB;
-  a.LS = g1.LS;
-  a.LB = g1.LB;
-  a.SBL = l0.SB;
-  a.LSL = l0.LS;
-  a.LBL = l0.LB;
-  a.n_long_items = int(long_items);
-  a.glinks = glink_total > 0 ? h->glinks.as<uint2>() : nullptr;
-  a.gflags = h->gflags.as<int>();
-  a.gdone = h->gflags.as<int>() + nflags;
-  a.lofs = db->dlofs.as<int64_t>();
-  a.links = (nlong_max > 0 && max_lstrips > 1) ? h->bbuf_long.as<uint2>() : nullptr;
-  a.lcap = lcap;
-  a.stream = db->stream.as<uint16_t>();
-  a.pairs = db->dpairs.as<PairRec>();
-  a.pair_end = np;
-  a.bbuf = (max_strips > 1 && min_pb < np) ? h->bbuf.as<uint2>() : nullptr;
-  a.bcap = bcap;
-  a.work_counter = h->counters.as<int>();
-  a.scores_all = c.dscores;
-  a.n_seqs = db->out_n;
-  a.thr = c.thr;
-  a.ovf = c.ovf;
-  a.ovf_count = c.ovf_count;
-  a.ovf_cap = int(c.ovf_cap);
-  a.code_pad2 = uint32_t(alpha) | (uint32_t(alpha) << 8);
-  a.nGe = c.nGe;
-  a.nGsGe = c.nGsGe;
-  auto* ev = c.timing ? next_event_pair(h) : nullptr;
-  if (ev) {
-    h->event_kind[h->n_events_used - 1] = 0;
-    SW_CK(cudaEventRecord(ev->first, c.st));
+  SW_CK(h->counters.ensure(3 * sizeof(int)));
+  SW_CK(cudaMemsetAsync(h->counters.p, 0, 3 * sizeof(int), c.st));
+  int* counters = h->counters.as<int>();
+  const uint32_t code_pad2 = uint32_t(alpha) | (uint32_t(alpha) << 8);
+
+  // ---- launches.  Long items: the long-pair kernel.  With short work too it runs
+  // concurrently on the handle's side stream (high priority), one CTA per SM (its
+  // shared-memory request leaves no room for a short-pair CTA, so co-resident short
+  // warps cannot stretch the longest pairs' critical path); the caller's stream
+  // waits for it (fork / join events), so the search stays stream-ordered.
+  const bool has_short = n_items1 > 0 || n_items0 > 0;
+  const bool fork = long_items > 0 && has_short && !combined;
+  LongArgs al{};
+  int smem_long = 0;
+  if (long_items > 0) {
+    const ProfGeom& l0 = gl[size_t(std::find_if(qnlong.begin(), qnlong.end(), [](int v) { return v > 0; }) -
+                                   qnlong.begin())];
+    al.queries = d_ldesc;
+    al.n_queries = int(ldesc.size());
+    al.n_items = int(long_items);
+    al.SBL = l0.SB; al.LSL = l0.LS; al.LBL = l0.LB;
+    smem_long = (W - 1) * LONG_RING * int(sizeof(uint2)) + W * l0.SB;
+    al.wcap = max_long + 64 + 8;
+    al.stream = db->stream.as<uint16_t>();
+    al.pairs = db->dpairs.as<PairRec>();
+    al.work_counter = counters + (combined ? 0 : 2);
+    al.thr = c.thr;
+    al.ovf = c.ovf;
+    al.ovf_count = c.ovf_count;
+    al.ovf_cap = int(c.ovf_cap);
+    al.code_pad2 = code_pad2;
+    al.nGe = c.nGe;
+    al.nGsGe = c.nGsGe;
   }
-  SW_CK(launch_inter(G, R, NT, grid, smem, a, c.st, wide0));
-  if (ev) SW_CK(cudaEventRecord(ev->second, c.st));
-  ++launches;
-  ++h->stats.n_score_launches;
-  h->stats.last_G = G;
-  h->stats.last_R = R;
+  if (long_items > 0 && !combined) {
+    int smem = smem_long;
+    if (fork) smem = std::max(smem, 200 * 1024);  // SM-exclusive (see above)
+    const int occ = long_max_ctas_per_sm(smem);
+    if (occ <= 0) fail(SW_ECUDA, "long-pair kernel does not fit on an SM");
+    const int grid = int(std::max<int64_t>(1, std::min<int64_t>(long_items, int64_t(occ) * h->sms)));
+    SW_CK(h->wrap.ensure(size_t(grid) * al.wcap * sizeof(uint2)));
+    al.wrap = h->wrap.as<uint2>();
+    cudaStream_t lst = c.st;
+    if (fork) {
+      if (!h->side) {
+        int lo_p = 0, hi_p = 0;
+        SW_CK(cudaDeviceGetStreamPriorityRange(&lo_p, &hi_p));
+        SW_CK(cudaStreamCreateWithPriority(&h->side, cudaStreamNonBlocking, hi_p));
+        SW_CK(cudaEventCreateWithFlags(&h->ev_fork, cudaEventDisableTiming));
+        SW_CK(cudaEventCreateWithFlags(&h->ev_join, cudaEventDisableTiming));
+      }
+      SW_CK(cudaEventRecord(h->ev_fork, c.st));
+      SW_CK(cudaStreamWaitEvent(h->side, h->ev_fork, 0));
+      lst = h->side;
+    }
+    std::pair<cudaEvent_t, cudaEvent_t>* ev = nullptr;
+    record_begin(h, c.timing, 1, lst, ev);
+    SW_CK(launch_long(grid, smem, al, lst));
+    if (ev) SW_CK(cudaEventRecord(ev->second, lst));
+    if (fork) SW_CK(cudaEventRecord(h->ev_join, lst));
+    ++out.launches;
+    ++h->stats.n_score_launches;
+  }
+  for (int mode : {1, 0}) {
+    const int n_short = mode == 1 ? n_items1 : n_items0;
+    if (n_short == 0) continue;
+    const int G = mode == 1 ? G1 : G0, R = mode == 1 ? R1 : R0;
+    ShortArgs as{};
+    as.slots = d_slots;
+    as.n_slots = int(sdesc.size());
+    as.n_items = n_short;
+    as.item_map = h->imap.as<int2>() + (mode == 1 ? 0 : n_items1);
+    int smem = 0;
+    if (mode == 1) {
+      as.SB = SB2; as.LS = LS2; as.LB = LB2;
+      as.ncopy = ncopy2;
+      as.cstride = SB2 + (ncopy2 > 1 ? 128 / ncopy2 : 0);
+      as.cskew = 0;
+      // two TMA-staged buffers (strip s and the prefetched strip s+1), 128-byte aligned
+      smem = 2 * ((((ncopy2 - 1) * as.cstride + SB2) + 127) / 128 * 128);
+    } else {
+      const Mode0Copies mc0 = mode0_copies(G, R, g0.LB, g0.SB, bank_copy, h->opt_bank_skew != 0);
+      as.SB = g0.SB; as.LS = g0.LS; as.LB = g0.LB;
+      as.ncopy = mc0.ncopy;
+      as.cstride = mc0.cstride;
+      as.cskew = mc0.skew;
+      smem = mc0.bytes;
+    }
+    const bool with_long = combined && mode == 0;
+    if (with_long) smem = std::max(smem, smem_long);  // an item is short or long: the two uses share smem
+    const int occ = with_long ? combined_max_ctas_per_sm(G, R, smem) : short_max_ctas_per_sm(mode, G, R, smem);
+    if (occ <= 0) fail(SW_ECUDA, "short-pair kernel does not fit on an SM");
+    const int64_t items = int64_t(n_short) + (with_long ? long_items : 0);
+    const int grid = int(std::max<int64_t>(1, std::min<int64_t>(items, int64_t(occ) * h->sms)));
+    const int min_pb = mode == 1 ? min_pb1 : min_pb0, max_strips = mode == 1 ? max_strips1 : max_strips0;
+    const int32_t max_short = min_pb < np ? db->pairs[size_t(min_pb)].len : 0;
+    as.bcap = ((max_short + 4 * G + 8 + 4) + 3) / 4 * 4;  // wave width up to V*G sub-lanes + align pad
+    DevBuf& bbuf = mode == 1 ? h->bbuf1 : h->bbuf0;
+    if (max_strips > 1) SW_CK(bbuf.ensure(size_t(grid) * (NT / G) * as.bcap * sizeof(uint2)));
+    as.bbuf = max_strips > 1 ? bbuf.as<uint2>() : nullptr;
+    as.stream = db->stream.as<uint16_t>();
+    as.pairs = db->dpairs.as<PairRec>();
+    as.pair_end = np;
+    as.work_counter = counters + mode;
+    as.scores_all = c.dscores;
+    as.n_seqs = db->out_n;
+    as.thr = c.thr;
+    as.ovf = c.ovf;
+    as.ovf_count = c.ovf_count;
+    as.ovf_cap = int(c.ovf_cap);
+    as.code_pad2 = code_pad2;
+    as.nGe = c.nGe;
+    as.nGsGe = c.nGsGe;
+    std::pair<cudaEvent_t, cudaEvent_t>* ev = nullptr;
+    record_begin(h, c.timing, 0, c.st, ev);
+    if (with_long) {
+      SW_CK(h->wrap.ensure(size_t(grid) * al.wcap * sizeof(uint2)));
+      al.wrap = h->wrap.as<uint2>();
+      SW_CK(launch_combined(G, R, grid, smem, as, al, c.st));
+    } else {
+      SW_CK(launch_short(mode, G, R, grid, smem, as, c.st));
+    }
+    if (ev) SW_CK(cudaEventRecord(ev->second, c.st));
+    ++out.launches;
+    ++h->stats.n_score_launches;
+    h->stats.last_G = G;
+    h->stats.last_R = R;
+  }
+  if (fork) SW_CK(cudaStreamWaitEvent(c.st, h->ev_join, 0));
 }
 
 int32_t sw_search(sw_handle_t h, const uint8_t* q_codes, const int64_t* q_offsets, int32_t n_queries, sw_db_t db,
@@ -1038,7 +1042,6 @@ int32_t sw_search(sw_handle_t h, const uint8_t* q_codes, const int64_t* q_offset
     SW_CK(h->ovf.ensure(size_t(std::max<int64_t>(ovf_cap, 1)) * sizeof(OvfRec)));
     SW_CK(h->ovf_count.ensure(sizeof(int)));
     SW_CK(cudaMemsetAsync(h->ovf_count.p, 0, sizeof(int), st));
-    const double sum_short = db->sum_short_len;
     const int32_t max_short = db->max_short, max_long = db->max_long;
     const uint32_t nGe16 = uint32_t(uint16_t(int16_t(-gap_extend)));
     const uint32_t nGsGe16 = uint32_t(uint16_t(int16_t(-(gap_open + gap_extend))));
@@ -1054,12 +1057,10 @@ int32_t sw_search(sw_handle_t h, const uint8_t* q_codes, const int64_t* q_offset
     lc.nGe = nGe16 | (nGe16 << 16);
     lc.nGsGe = nGsGe16 | (nGsGe16 << 16);
     lc.timing = timing;
-    lc.sum_short = sum_short;
-    lc.max_short = max_short;
-    lc.max_long = max_long;
-    double cells_computed = 0;
+    LaunchOut lo;
     const uint8_t* dq = h->qcodes.as<uint8_t>();
-    launch_all(lc, qlen, qoff0, cells_computed, launches);
+    launch_all(lc, qlen, qoff0, lo);
+    launches += lo.launches;
     if (ovf_cap > 0) {
       // Exact int32 re-score of the flagged pairs, enqueued unconditionally: the
       // kernel reads the flagged count on the device and exits at once when it is
@@ -1122,9 +1123,8 @@ int32_t sw_search(sw_handle_t h, const uint8_t* q_codes, const int64_t* q_offset
     double sq = 0;
     for (auto L : qlen) sq += double(L);
     h->stats.cells = sq * double(db->n_res);
-    const double short_res = db->short_res;
-    h->stats.cells_short = sq * short_res;  // pairs <= 3000 columns (inter-task mode)
-    h->stats.cells_computed = cells_computed;
+    h->stats.cells_short = lo.cells_short;  // scored by the short-pair (inter-task) kernels
+    h->stats.cells_computed = lo.cells_computed;
     h->stats.n_launches = launches;
   });
 }
@@ -1458,8 +1458,9 @@ int32_t sw_free(sw_handle_t h) {
     cudaEventDestroy(e.first);
     cudaEventDestroy(e.second);
   }
-  for (cudaEvent_t e : {h->ev_begin, h->ev_end})
+  for (cudaEvent_t e : {h->ev_begin, h->ev_end, h->ev_fork, h->ev_join})
     if (e) cudaEventDestroy(e);
+  if (h->side) cudaStreamDestroy(h->side);
   if (h->ev_done) cudaEventDestroy(h->ev_done);
   delete h;
   return SW_OK;

@@ -1,11 +1,14 @@
-// SWDUAL hot-path kernels for sm_100a: query-profile build, the inter-task
-// s16x2 DPX scoring kernel and the exact int32 re-score kernel.
+// SWDUAL hot-path kernels for sm_100a: query-profile builds, the inter-task
+// s16x2 DPX scoring kernels (short pairs), the intra-task chained-warp kernel
+// (long pairs), the exact int32 re-score, the mapped-output zeroing and the
+// gathered-block merge.
 //
-// Inter-task kernel (the paper's "very coarse-grained" split
+// Inter-task kernels (the paper's "very coarse-grained" split
 // across workers, with the "fine-grained" wavefront inside a
 // worker, L202-216 / Fig. 2):
 //   * a lane GROUP of G lanes scores one database pair (two length-neighbours,
-//     one per s16x2 half) against one query;
+//     one per s16x2 half) against one query (mode 0), or one database sequence
+//     against a query PAIR (mode 1, two queries per s16x2 register);
 //   * lane k of the group owns R consecutive query rows of the current strip
 //     (strip height G*R rows); at step t it computes column t-k, so the group
 //     sweeps the matrix as an anti-diagonal wave: the bottom row (H, F) and the
@@ -13,9 +16,11 @@
 //   * queries taller than one strip are done in passes; the last lane writes the
 //     strip's bottom row to a per-group global boundary row that lane 0 reads
 //     in the next pass;
-//   * the int8 query profile of the current strip sits in shared memory;
+//   * the query profile of the current strip sits in shared memory;
 //   * CTAs are persistent and take chunks of NT/G pairs from an atomic counter,
 //     pairs sorted longest first.
+// Each mode is its own kernel (its own register budget: the query-pair kernel
+// holds 2 CTAs per SM at 128 registers with R up to 32).
 #include <algorithm>
 #include <cstdio>
 #include "sw_internal.h"
@@ -27,13 +32,7 @@ constexpr int8_t PAD_SCORE = -64;  // S[.][PAD] = S[PAD][.] <= 0 (reading R-12)
 // Intra-task mode: a strip starts consuming the row above only once its
 // producer is this many columns ahead, so producer and consumer warps of a
 // chain run decoupled instead of in lock-step (the consumer then rarely waits).
-constexpr int LINK_LAG = 64;
-#ifndef SW_DUAL_LONG
-#define SW_DUAL_LONG 0
-#endif
-#ifndef SW_DUAL
-#define SW_DUAL 1  // both sub-lanes in one interleaved row sweep (gotoh_rows_dual)
-#endif
+constexpr int LINK_LAG = 32;
 constexpr int RESCORE_LAG = 16;  // re-score chains: one round per CTA, short lag keeps the critical path short
 
 // ---------------------------------------------------------------------------
@@ -100,7 +99,7 @@ __global__ void build_profile_q2_kernel(const uint8_t* __restrict__ qa, int ma, 
         // rows past a query, and PAD codes (= alpha) that pad packed queries to whole strips
         const int ca = row < ma ? qa[row] : alpha, cb = row < mb ? qb[row] : alpha;
         const int va = (ca < alpha && a < alpha) ? M[ca * alpha + a] : PAD_SCORE;
-        const int vb = mb < 0 ? 0 : (cb < alpha && a < alpha) ? M[cb * alpha + a] : PAD_SCORE;  // mb < 0: wide mode-0 profile
+        const int vb = (cb < alpha && a < alpha) ? M[cb * alpha + a] : PAD_SCORE;
         v = (uint32_t(va) & 0xffffu) | (uint32_t(vb) << 16);
       }
     }
@@ -139,65 +138,6 @@ __device__ __forceinline__ int copy_off(int cp, int csx, uint32_t skew) {
   return cp * csx + 4 * int((skew >> (8 * cp)) & 0xffu);
 }
 
-// DB codes of the current pair: every strip pass of an item re-reads them, so
-// they could stay cached between strips (SW_CODES 0: streaming/evict-first,
-// 1: default caching, 2: L2 evict_last).  Measured on config 3: 1 and 2 cut
-// DRAM reads by 23% but run 1% slower (the kernel is ALU-bound); 0 is kept.
-#ifndef SW_CODES
-#define SW_CODES 0
-#endif
-// SW_Q2_ADDR 1: lane 0 turns the DB letter into its profile-row address once per
-// column (PRMT + IMAD) and the lanes shuffle addresses instead of codes: 2 fewer
-// ALU ops per column, but the extra live register doubles the spill at the
-// 128-register cap -- measured -7.5% on config 3 (+0.4% on config 2); kept off.
-// SW_SEL_IMAD 1: lane 0's three per-column selects (code, H, F of the row above)
-// as integer multiply-adds (FMA pipe) instead of SEL (ALU pipe).  Measured -2% on
-// config 3 (+0.8% on config 4): one ALU op traded for two issue slots; kept off.
-// SW_T0_UNROLL: unroll factor of the 4-column block loop of a strip pass (2 measured
-// -1.4% on config 3: more register moves and spill; kept at 1)
-#ifndef SW_T0_UNROLL
-#define SW_T0_UNROLL 1
-#endif
-#ifndef SW_SEL_IMAD
-#define SW_SEL_IMAD 0
-#endif
-// a == 1 ? v : x, as x + a * (v - x) in two IMADs (a in {0, 1}; exact mod 2^32)
-__device__ __forceinline__ uint32_t fma_sel(uint32_t a, uint32_t v, uint32_t x) {
-  uint32_t d, r;
-  asm("mad.lo.u32 %0, %1, 1, %2;" : "=r"(d) : "r"(v), "r"(0u - x));
-  asm("mad.lo.u32 %0, %1, %2, %3;" : "=r"(r) : "r"(a), "r"(d), "r"(x));
-  return r;
-}
-#ifndef SW_Q2_ADDR
-#define SW_Q2_ADDR 0
-#endif
-#ifndef SW_BB_HINT
-#define SW_BB_HINT 0
-#endif
-__device__ __forceinline__ uint4 ld_bb(const uint2* p, uint64_t pol) {
-  if constexpr (SW_BB_HINT) return ld_l2_last(p, pol);
-  else return *reinterpret_cast<const uint4*>(p);
-}
-__device__ __forceinline__ void st_bb(uint2* p, uint2 v, uint64_t pol) {
-  if constexpr (SW_BB_HINT) st_l2_last(p, v, pol);
-  else *p = v;
-}
-__device__ __forceinline__ uint2 ld_codes(const uint2* p, uint64_t pol) {
-  if constexpr (SW_CODES == 0) return __ldcs(p);
-  else if constexpr (SW_CODES == 1) return __ldg(p);
-  else {
-    uint2 v;
-    asm volatile("ld.global.nc.L2::cache_hint.v2.u32 {%0, %1}, [%2], %3;" : "=r"(v.x), "=r"(v.y) : "l"(p), "l"(pol));
-    return v;
-  }
-}
-
-// One strip pass of a lane group over one pair: G lanes x R rows, columns
-// streamed as an anti-diagonal wave.  Boundary rows: lane 0 reads the strip
-// above at rp[c] (c = column, rp = row base + G - 1), lane G-1 writes this
-// strip's bottom row at wp[t] (t = step).  LINKED: the row above is produced
-// concurrently by another warp of the CTA (intra-task mode): lane 0 waits on
-// its progress counter, lane G-1 publishes its own.
 template <int R>
 struct SubLanes {
   // Each lane runs V "sub-lanes" of R/V rows, the second one column behind the
@@ -206,13 +146,50 @@ struct SubLanes {
   static constexpr int V = (R % 8 == 0) ? 2 : 1;
 };
 
-template <int G, int R, bool LINKED, bool Q2 = false, int US = (Q2 ? 16 : ((R % 8 == 0) ? 8 : 4)), int PW = 0>
+// Boundary cells of a strip pass.  Short items: a per-group row in global memory
+// (written in one pass, read in the next).  Long items: a shared-memory ring
+// between two concurrently running warps (producer progress / consumer progress
+// counters, LONG_RING steps of slack) or, for the round wrap, a global row.
+struct Chain {
+  bool in_ring, out_ring;    // rings (shared memory) or global rows
+  uint32_t in_sring, out_sring;  // shared-window addresses of the rings
+  int* in_prog;              // producer progress (steps written, monotone across rounds), shared
+  int* in_cons;              // this warp's consumption of its input, published for the producer
+  int* out_prog;             // this warp's output progress
+  const int* out_cons;       // consumption of this warp's output by its consumer
+  int in_base, out_base;     // step index (monotone across rounds) of the producer's / this warp's step 0
+  const uint2* grow_in;      // global input row (round wrap)
+  uint2* grow_out;           // global output row (round wrap)
+};
+
+__device__ __forceinline__ uint4 lds128v(uint32_t a) { return lds128(a); }
+__device__ __forceinline__ void sts64(uint32_t a, uint2 v) {
+  asm volatile("st.shared.v2.u32 [%0], {%1, %2};" :: "r"(a), "r"(v.x), "r"(v.y) : "memory");
+}
+
+// Warp-uniform spin until *p >= need: lane `who` (the lane whose later shared
+// memory accesses the counter orders) polls with acquire, the value is broadcast.
+__device__ __forceinline__ void wait_geq(const int* p, int need, int& seen, int who) {
+  if (seen >= need) return;
+  for (;;) {
+    int v = 0;
+    if ((threadIdx.x & 31) == who) v = ld_acquire_cta(p);
+    v = __shfl_sync(FULL, v, who);
+    if (v >= need) { seen = v; return; }
+    __nanosleep(32);
+  }
+}
+
+// One strip pass of a lane group over one pair: G lanes x R rows, columns
+// streamed as an anti-diagonal wave.  Boundary rows: lane 0 reads the strip
+// above at rp[c] (c = column, rp = row base + G - 1), lane G-1 writes this
+// strip's bottom row at wp[t] (t = step).  LINKED (long items, G = 32): the
+// row above is produced concurrently by another warp of the CTA (Chain).
+template <int G, int R, bool LINKED, bool Q2 = false, int US = (Q2 ? 16 : ((R % 8 == 0) ? 8 : 4))>
 __device__ __forceinline__ void strip_pass(const uint8_t* sprof, int LS, int LB, const uint16_t* pstream, int L,
                                            int T, int k, bool rd, bool wr, const uint2* __restrict__ rp,
-                                           uint2* __restrict__ wp, const Link& lk, uint32_t code_pad2,
-                                           uint32_t nGe, uint32_t nGsGe, uint32_t& best, uint32_t shift = 0,
-                                           uint32_t wmul = 0) {
-  static_assert(!PW || (!Q2 && R % 8 == 0 && US == 16), "wide single-query profile: two sub-lanes, LDS.128 rows");
+                                           uint2* __restrict__ wp, const Chain& ch, uint32_t code_pad2,
+                                           uint32_t nGe, uint32_t nGsGe, uint32_t& best, uint32_t shift = 0) {
   constexpr int V = SubLanes<R>::V;
   constexpr int VG = V * G;   // width of the wave in sub-lanes
   constexpr int RH = R / V;   // rows per sub-lane
@@ -220,64 +197,68 @@ __device__ __forceinline__ void strip_pass(const uint8_t* sprof, int LS, int LB,
 #pragma unroll
   for (int r = 0; r < R; ++r) { HA[r] = 0; E[r] = 0; }
   const uint32_t sbase = static_cast<uint32_t>(__cvta_generic_to_shared(sprof));
-  // Q2 (SW_Q2_ADDR): the code that travels down the lanes is already the shared
-  // address of the DB letter's profile row (lane-independent); lane 0 forms it
-  // once per column with one PRMT (byte select) + IMAD, the others add laneoff.
-  const uint32_t c0pad = (Q2 && SW_Q2_ADDR) ? sbase + (code_pad2 & 0xffu) * LS : code_pad2;
-  uint32_t hdiag = 0, sH = 0, sF = 0, sC = c0pad;
+  uint32_t hdiag = 0, sH = 0, sF = 0, sC = code_pad2;
   const uint2* __restrict__ codes = reinterpret_cast<const uint2*>(pstream);
   const uint32_t pad4 = code_pad2 | (code_pad2 << 16);
   const uint32_t laneoff = uint32_t(k) * LB;
   const bool lead = (k == 0), tail = (k == G - 1);
-#if SW_SEL_IMAD
-  const uint32_t lead01 = lead ? 1u : 0u;
-#endif
   const uint2 z2 = make_uint2(0, 0);
   // second sub-lane: its inputs are the first sub-lane's outputs of the previous step
-  uint32_t hdiag1 = 0, cH = 0, cF = 0, pC = c0pad;
-  const uint32_t bsel = (shift >> 3) | 0x4440u;  // PRMT selector: byte `shift/8` of a column word, zero-extended
+  uint32_t hdiag1 = 0, cH = 0, cF = 0, pC = code_pad2;
   const uint32_t pad_row = sbase + (code_pad2 & 0xffu) * LS + laneoff;
   uint32_t ppa = pad_row, ppb = pad_row;
-  rp += VG - 1;  // sub-lane 0 of lane 0 reads column c at rp[c + VG - 1]
-  // SW_BB_HINT 1: boundary rows with an L2 evict_last policy (DRAM writes -35%
-  // on config 3, but 1% slower: the kernel is ALU-bound, DRAM is ~3% busy)
-  const uint64_t pol = (SW_BB_HINT || SW_CODES == 2) ? l2_evict_last_policy() : 0;
+  // input index of sub-lane 0 of lane 0 for column c: c + VG - 1 (producer step)
+  const int ioff = VG - 1;
+  int seen_in = -1, seen_out = -1;
 
   // lane 0 prefetch of block 0: 4 columns of codes and (if rd) 4 boundary cells.
   // L and t0 are multiples of 4, so one compare guards a whole block.
-  uint2 cw = make_uint2(pad4, pad4);
-  uint2 tb0 = z2, tb1 = z2, tb2 = z2, tb3 = z2;
-  int seen = -1;
-  if (LINKED && rd && L > 0) wait_progress(lk, lk.in_base + min(4 + VG - 1 + LINK_LAG, L + VG), seen);
-  if (lead && L > 0) {
-    cw = ld_codes(codes, pol);
+  auto load_block = [&](int t0, uint2& cw, uint2& b0, uint2& b1, uint2& b2, uint2& b3) {
+    cw = __ldcs(codes + (t0 >> 2));
     if (rd) {
-      if (LINKED) { tb0 = __ldcg(rp + 0); tb1 = __ldcg(rp + 1); tb2 = __ldcg(rp + 2); tb3 = __ldcg(rp + 3); }
-      else {  // rp is 32-byte aligned (see the bb base in inter_kernel)
-        const uint4 x = ld_bb(rp, pol), y = ld_bb(rp + 2, pol);
-        tb0 = make_uint2(x.x, x.y); tb1 = make_uint2(x.z, x.w); tb2 = make_uint2(y.x, y.y); tb3 = make_uint2(y.z, y.w);
+      if constexpr (LINKED) {
+        if (ch.in_ring) {
+          const int x = ch.in_base + t0 + ioff;  // 3 mod 4 (ioff = 63): the 4 cells one by one
+          const uint32_t a0 = ch.in_sring + uint32_t((x & (LONG_RING - 1)) * 8);
+          const uint32_t a1 = ch.in_sring + uint32_t(((x + 1) & (LONG_RING - 1)) * 8);
+          const uint32_t a2 = ch.in_sring + uint32_t(((x + 2) & (LONG_RING - 1)) * 8);
+          const uint32_t a3 = ch.in_sring + uint32_t(((x + 3) & (LONG_RING - 1)) * 8);
+          b0 = lds64(a0); b1 = lds64(a1); b2 = lds64(a2); b3 = lds64(a3);
+        } else {
+          const uint2* g = ch.grow_in + t0 + ioff;
+          b0 = __ldcg(g); b1 = __ldcg(g + 1); b2 = __ldcg(g + 2); b3 = __ldcg(g + 3);
+        }
+      } else {  // rp is 32-byte aligned at rp + ioff (see the bb base in short_body)
+        const uint4 x = *reinterpret_cast<const uint4*>(rp + t0 + ioff);
+        const uint4 y = *reinterpret_cast<const uint4*>(rp + t0 + ioff + 2);
+        b0 = make_uint2(x.x, x.y); b1 = make_uint2(x.z, x.w); b2 = make_uint2(y.x, y.y); b3 = make_uint2(y.z, y.w);
       }
     }
+  };
+  // long items: progress this warp's consumer needs before block t0's prefetch
+  auto wait_in = [&](int t0) {
+    if constexpr (LINKED) {
+      if (rd) wait_geq(ch.in_prog, ch.in_base + min(t0 + 4 + ioff + LINK_LAG, L + VG), seen_in, 0);
+    }
+  };
+  uint2 cw = make_uint2(pad4, pad4);
+  uint2 tb0 = z2, tb1 = z2, tb2 = z2, tb3 = z2;
+  if (L > 0) {
+    wait_in(0);
+    if (lead) load_block(0, cw, tb0, tb1, tb2, tb3);
   }
   __syncwarp();
-#if SW_T0_UNROLL == 2
-#pragma unroll 2
-#endif
   for (int t0 = 0; t0 < T; t0 += 4) {
     const uint2 cwc = cw;
     const uint2 c0 = tb0, c1 = tb1, c2 = tb2, c3 = tb3;
-    rp += 4;
-    if (LINKED && rd && t0 + 4 < L) wait_progress(lk, lk.in_base + min(t0 + 8 + VG - 1 + LINK_LAG, L + VG), seen);
+    if (t0 + 4 < L) wait_in(t0 + 4);
+    if constexpr (LINKED) {
+      // ring space for this block's outputs (the consumer may lag by up to LONG_RING steps)
+      if (wr && ch.out_ring) wait_geq(ch.out_cons, ch.out_base + t0 + 4 - LONG_RING, seen_out, G - 1);
+    }
     if (lead) {
       if (t0 + 4 < L) {
-        cw = ld_codes(codes + ((t0 + 4) >> 2), pol);
-        if (rd) {
-          if (LINKED) { tb0 = __ldcg(rp + 0); tb1 = __ldcg(rp + 1); tb2 = __ldcg(rp + 2); tb3 = __ldcg(rp + 3); }
-          else {
-            const uint4 x = ld_bb(rp, pol), y = ld_bb(rp + 2, pol);
-            tb0 = make_uint2(x.x, x.y); tb1 = make_uint2(x.z, x.w); tb2 = make_uint2(y.x, y.y); tb3 = make_uint2(y.z, y.w);
-          }
-        }
+        load_block(t0 + 4, cw, tb0, tb1, tb2, tb3);
       } else {
         cw = make_uint2(pad4, pad4);
         tb0 = z2; tb1 = z2; tb2 = z2; tb3 = z2;
@@ -289,30 +270,15 @@ __device__ __forceinline__ void strip_pass(const uint8_t* sprof, int LS, int LB,
       uint32_t rH = __shfl_up_sync(FULL, sH, 1, G);
       uint32_t rF = __shfl_up_sync(FULL, sF, 1, G);
       uint32_t rC = __shfl_up_sync(FULL, sC, 1, G);
-#if SW_SEL_IMAD
-      {  // lane 0 takes the boundary row: x + lead01 * (v - x) on the FMA pipe instead of SEL (ALU)
-        const uint32_t w = (j < 2) ? cwc.x : cwc.y;
-        const uint32_t cl = (j & 1) ? (w >> 16) : (w & 0xffffu);
-        const uint2 tv = (j == 0) ? c0 : (j == 1) ? c1 : (j == 2) ? c2 : c3;
-        rC = fma_sel(lead01, cl, rC);
-        rH = fma_sel(lead01, tv.x, rH);
-        rF = fma_sel(lead01, tv.y, rF);
-      }
-#else
       if (lead) {
         const uint32_t w = (j < 2) ? cwc.x : cwc.y;
-        if constexpr (Q2 && SW_Q2_ADDR) rC = sbase + prmt(w, 0u, bsel + ((j & 1) ? 2u : 0u)) * LS;
-        else rC = (j & 1) ? (w >> 16) : (w & 0xffffu);
+        rC = (j & 1) ? (w >> 16) : (w & 0xffffu);
         const uint2 tv = (j == 0) ? c0 : (j == 1) ? c1 : (j == 2) ? c2 : c3;
         rH = tv.x;
         rF = tv.y;
       }
-#endif
       uint32_t pa, pb;
-      if constexpr (Q2 && SW_Q2_ADDR) {  // rC = profile-row address of the DB letter
-        pa = rC + laneoff;
-        pb = pa;
-      } else if constexpr (Q2) {  // one DB sequence (byte `shift` of the pair word) against two queries
+      if constexpr (Q2) {  // one DB sequence (byte `shift` of the pair word) against two queries
         pa = sbase + ((rC >> shift) & 0xffu) * LS + laneoff;
         pb = pa;
       } else {
@@ -321,9 +287,8 @@ __device__ __forceinline__ void strip_pass(const uint8_t* sprof, int LS, int LB,
       }
       if constexpr (V == 2) {
         uint32_t h1 = cH, f1 = cF;
-        if constexpr (SW_DUAL && (Q2 || PW || (SW_DUAL_LONG && LINKED))) {  // measured: +3% for the query-pair mode, -2% with the PRMT (mode 0)
-          gotoh_rows_dual<R, Q2, US, PW>(HA, E, best, hdiag, pa, pb, rH, rF, hdiag1, ppa, ppb, h1, f1, nGe, nGsGe,
-                                         wmul);
+        if constexpr (Q2) {  // measured: +3% for the query-pair mode, -2% with the PRMT (mode 0)
+          gotoh_rows_dual<R, Q2, US>(HA, E, best, hdiag, pa, pb, rH, rF, hdiag1, ppa, ppb, h1, f1, nGe, nGsGe);
         } else {
           // sub-lane 1 (rows RH..R-1, column t-1) first: it reads rows it owns only
           gotoh_rows_inplace<R, RH, R, Q2, US>(HA, E, best, hdiag1, ppa, ppb, h1, f1, nGe, nGsGe);
@@ -344,395 +309,437 @@ __device__ __forceinline__ void strip_pass(const uint8_t* sprof, int LS, int LB,
         sC = rC;
       }
       if (wr && tail) {
-        if (LINKED) __stcg(wp + j, make_uint2(sH, sF));
-        else st_bb(wp + j, make_uint2(sH, sF), pol);
-      }
-    }
-    wp += 4;
-    if (LINKED && wr && tail) {  // release orders this lane's link writes before the counter
-      if (!lk.out_gpu) st_release_cta(lk.out, lk.out_base + t0 + 4);
-      else if (((t0 >> 2) & 3) == 3 || t0 + 4 >= T) st_release_gpu(lk.out, lk.out_base + t0 + 4);
-    }
-  }
-}
-
-__device__ __forceinline__ void emit_pair(const InterArgs& a, const QueryDesc& d, int p, const PairRec& pr,
-                                          uint32_t best) {
-  const int lo = int(int16_t(best & 0xffffu));
-  const int hi = int(int16_t(best >> 16));
-  d.scores[pr.id0] = lo;
-  if (lo >= a.thr) {
-    const int e = atomicAdd(a.ovf_count, 1);
-    if (e < a.ovf_cap) a.ovf[e] = OvfRec{d.qidx, p, 0, 0};
-  }
-  if (pr.id1 >= 0) {
-    d.scores[pr.id1] = hi;
-    if (hi >= a.thr) {
-      const int e = atomicAdd(a.ovf_count, 1);
-      if (e < a.ovf_cap) a.ovf[e] = OvfRec{d.qidx, p, 1, 0};
-    }
-  }
-}
-
-// Persistent kernel over ALL queries of a search.  Work items, costliest first:
-//   [0, Q*n_long): (query, LONG pair) -- scored by all W = NT/32 warps of the CTA
-//     together (intra-task mode; the paper's fine-grained
-//     wavefront across PEs, Fig. 2): warp w takes strips w, w+W, ...
-//     of a 32-lane x LONG_R-row geometry, each strip consuming the bottom row of
-//     the strip above through a global link row + shared progress counter;
-//   then (query, CHUNK of NT/G short pairs) -- one pair per lane group
-//     (inter-task mode).
-// Queries are in descending length, pairs in descending length.
-// PWK = 1: the variant whose single-query slots use the wide profile (a separate
-// instantiation: its pair build needs more live registers, which must not raise
-// the register allocation of the default kernel).
-template <int G, int R, int NT, int PWK>
-__device__ __forceinline__ void inter_body(InterArgs a) {
-  extern __shared__ __align__(16) uint8_t smem[];
-  // An item is either short or long, so the two uses share shared memory:
-  uint8_t* sprof = smem;                         // short mode: the strip profile (bank-spread copies)
-  uint8_t* lprof = smem + (SW_SMEM_UNION ? 0 : max(a.cstride[0] * (a.ncopy[0] - 1) + 128 + a.SB,
-                                                    a.cstride[1] * (a.ncopy[1] - 1) + a.SB2));  // long mode: one a.SBL slot per warp
-  __shared__ int s_item;
-  __shared__ int s_prog[NT / 32];
-  __shared__ uint32_t s_best[NT / 32];
-  constexpr int NG = NT / G;
-  constexpr int W = NT / 32;
-  const int tid = threadIdx.x;
-  const int k = tid & (G - 1);
-  const int g = tid / G;
-  const int lane = tid & 31, warp = tid >> 5;
-  const int n_long_items = a.n_long_items;
-  const int n_items = n_long_items + a.n_short_items;
-  // per-group boundary row; offset so that &bb[V*G - 1] is 32-byte aligned (bcap % 4 == 0)
-  constexpr int BB_PAD = (4 - (G * SubLanes<R>::V - 1) % 4) % 4;
-  uint2* __restrict__ bb = a.bbuf + ((size_t)blockIdx.x * NG + g) * (size_t)a.bcap + BB_PAD;
-  int loaded = -1;  // (query rank << 16 | strip) of the short profile in shared memory (CTA-uniform)
-
-  for (;;) {
-    if (tid == 0) s_item = atomicAdd(a.work_counter, 1);
-    if (tid < W) { s_prog[tid] = -1; s_best[tid] = 0; }
-    __syncthreads();
-    const int item = s_item;
-    if (item >= n_items) break;
-    if (item < n_long_items) {
-      loaded = -1;  // the long-mode slots overwrite the short strip profile
-      // ---------------- long pair, superstrip k: W chained strips on this CTA's
-      // warps; superstrips k-1 / k+1 of the same pair run on other CTAs
-      int lo = 0, hi = a.n_queries - 1;
-      while (lo < hi) {
-        const int mid = (lo + hi + 1) >> 1;
-        if (a.queries[mid].long_item_begin <= item) lo = mid; else hi = mid - 1;
-      }
-      const QueryDesc d = a.queries[lo];
-      if (d.pairs_per_item > 1) {
-        // ---- query shorter than W strips: P = W / S pairs per CTA, S warps per
-        // pair (one strip each; upstream strips on higher warp ids)
-        const int S = d.n_strips_long, P = d.pairs_per_item;
-        const int grp = warp / S, jw = warp - grp * S;
-        const int pidx = (item - d.long_item_begin) * P + grp;
-        const bool active = grp < P && pidx < d.n_long;
-        uint32_t best = 0;
-        if (active) {
-          const PairRec pr = a.pairs[pidx];
-          const int s = S - 1 - jw;
-          uint8_t* myprof = lprof + warp * a.SBL;
-          {
-            const uint4* src = reinterpret_cast<const uint4*>(d.prof_long + (size_t)s * a.SBL);
-            uint4* dst = reinterpret_cast<uint4*>(myprof);
-            for (int i = lane; i < a.SBL / 16; i += 32) dst[i] = __ldg(src + i);
-          }
-          __syncwarp();
-          uint2* links = a.links + (size_t)blockIdx.x * W * a.lcap;
-          Link lk{};
-          const int wprod = warp + 1;  // the warp holding strip s-1 of this pair
-          lk.in = &s_prog[s > 0 ? wprod : warp];
-          lk.in_base = (s - 1) << 20;
-          lk.out = &s_prog[warp];
-          lk.out_base = s << 20;
-          strip_pass<32, LONG_R, true, false, LONG_US>(myprof, a.LSL, a.LBL, a.stream + pr.off, pr.len,
-                                       pr.len + 32 * SubLanes<LONG_R>::V, lane, s > 0, s + 1 < S,
-                                       links + (size_t)(s > 0 ? wprod : warp) * a.lcap,
-                                       links + (size_t)warp * a.lcap, lk, a.code_pad2, a.nGe, a.nGsGe, best);
-        }
-#pragma unroll
-        for (int o = 16; o > 0; o >>= 1) best = __vmaxs2(best, __shfl_xor_sync(FULL, best, o));
-        if (lane == 0) s_best[warp] = best;
-        __syncthreads();
-        if (tid < P) {
-          const int pj = (item - d.long_item_begin) * P + tid;
-          if (pj < d.n_long) {
-            uint32_t b = 0;
-            for (int w = tid * S; w < tid * S + S; ++w) b = __vmaxs2(b, s_best[w]);
-            emit_pair(a, d, pj, a.pairs[pj], b);
-          }
-        }
-        __syncthreads();
-        continue;
-      }
-      const int K = d.n_super;               // CTAs sharing this pair
-      const int64_t gstride = d.glink_stride;
-      const int local = item - d.long_item_begin;
-      const int pidx = local / K, c = local - pidx * K;
-      const PairRec pr = a.pairs[pidx];
-      const int T = pr.len + 32 * SubLanes<LONG_R>::V;
-      uint32_t best = 0;
-      uint8_t* myprof = lprof + warp * a.SBL;
-      uint2* links = a.links + (size_t)blockIdx.x * W * a.lcap;
-      uint2* grow = a.glinks + d.glink_base + a.lofs[pidx];
-      int* gflag = a.gflags + d.flag_base + (int64_t)pidx * K;
-      // Strips are dealt round-robin: round r of CTA c covers strips
-      // W*(K*r + c) .. +W-1, one per warp.  Upstream strips run on the HIGHER
-      // warp ids: the SMSP arbiter issues highest-warp-id first, so producers
-      // keep their lead instead of being starved by consumers that caught up
-      // and spin on the link counter.  The chain runs warp W-1 -> 0 inside a
-      // CTA, then on to CTA c+1 (global boundary row + GPU-scope counter), and
-      // from CTA K-1 back to CTA 0 for the next round.
-      const int j = W - 1 - warp;
-      const int ns = d.n_strips_long;
-      for (int r = 0;; ++r) {
-        const int s = W * (K * r + c) + j;   // strip index
-        if (s >= ns) break;
-        __syncwarp();
-        {  // this warp's strip profile -> its own slot
-          const uint4* src = reinterpret_cast<const uint4*>(d.prof_long + (size_t)s * a.SBL);
-          uint4* dst = reinterpret_cast<uint4*>(myprof);
-          for (int i = lane; i < a.SBL / 16; i += 32) dst[i] = __ldg(src + i);
-        }
-        __syncwarp();
-        const bool rd = s > 0, wr = s + 1 < ns;
-        Link lk{};
-        const uint2* rp;
-        uint2* wp;
-        if (j > 0 || K == 1) {  // producer is a warp of this CTA (for K == 1: the last warp, previous round)
-          const int jl = (j + W - 1) % W;
-          rp = links + (size_t)jl * a.lcap;
-          lk.in = &s_prog[jl];
-        } else {                // producer is the last warp of CTA c-1 (or of CTA K-1, previous round)
-          const int pc = (c + K - 1) % K;
-          rp = grow + (int64_t)pc * gstride;
-          lk.in = gflag + pc;
-          lk.in_gpu = true;
-        }
-        lk.in_base = (s - 1) << 20;  // counters are monotone: (strip << 20) | cells written
-        if (j < W - 1 || K == 1) {
-          wp = links + (size_t)j * a.lcap;
-          lk.out = &s_prog[j];
+        if constexpr (LINKED) {
+          if (ch.out_ring) sts64(ch.out_sring + uint32_t(((ch.out_base + t0 + j) & (LONG_RING - 1)) * 8), make_uint2(sH, sF));
+          else __stcg(ch.grow_out + t0 + j, make_uint2(sH, sF));
         } else {
-          wp = grow + (int64_t)c * gstride;
-          lk.out = gflag + c;
-          lk.out_gpu = true;
-        }
-        lk.out_base = s << 20;
-        strip_pass<32, LONG_R, true, false, LONG_US>(myprof, a.LSL, a.LBL, a.stream + pr.off, pr.len, T, lane, rd, wr, rp, wp, lk,
-                                     a.code_pad2, a.nGe, a.nGsGe, best);
-      }
-#pragma unroll
-      for (int o = 16; o > 0; o >>= 1) best = __vmaxs2(best, __shfl_xor_sync(FULL, best, o));
-      if (lane == 0) s_best[warp] = best;
-      __syncthreads();
-      if (tid == 0) {
-        uint32_t b = 0;
-        for (int w = 0; w < W; ++w) b = __vmaxs2(b, s_best[w]);
-        if (K == 1) {
-          emit_pair(a, d, pidx, pr, b);
-        } else {  // combine the superstrips' maxima; the last one to finish checks overflow
-          atomicMax(d.scores + pr.id0, int(int16_t(b & 0xffffu)));
-          if (pr.id1 >= 0) atomicMax(d.scores + pr.id1, int(int16_t(b >> 16)));
-          __threadfence();
-          if (atomicAdd(a.gdone + d.done_base + pidx, 1) == K - 1) {
-            __threadfence();
-            const int v0 = atomicAdd(d.scores + pr.id0, 0);
-            const int v1 = pr.id1 >= 0 ? atomicAdd(d.scores + pr.id1, 0) : 0;
-            if (v0 >= a.thr) {
-              const int e = atomicAdd(a.ovf_count, 1);
-              if (e < a.ovf_cap) a.ovf[e] = OvfRec{d.qidx, pidx, 0, 0};
-            }
-            if (pr.id1 >= 0 && v1 >= a.thr) {
-              const int e = atomicAdd(a.ovf_count, 1);
-              if (e < a.ovf_cap) a.ovf[e] = OvfRec{d.qidx, pidx, 1, 0};
-            }
-          }
-        }
-      }
-    } else {
-      // ---------------- short work: the host ordered all (slot, chunk) items of
-      // the launch by critical path (strips x pair length), longest first
-      const int2 sc = a.item_map[item - n_long_items];
-      const int sl = sc.x;
-      const SlotDesc d = a.slots[sl];
-      const int chunk = sc.y;
-      const bool q2 = d.mode == 1;
-      constexpr bool wide = PWK != 0 && R % 8 == 0;  // mode 0 with the 32-bit (query-pair layout) profile
-      int p, half = 0;
-      if (q2) {  // chunk of NG half-pairs: DB sequence = one half of a pair
-        const int hp = chunk * NG + g;
-        p = d.pair_begin + (hp >> 1);
-        half = hp & 1;
-      } else {
-        p = d.pair_begin + chunk * NG + g;
-      }
-      bool valid = p < a.pair_end;
-      PairRec pr;
-      if (valid) pr = a.pairs[p];
-      else { pr.off = 0; pr.len = 0; pr.id0 = -1; pr.id1 = -1; }
-      if (q2 && half && pr.id1 < 0) valid = false;  // odd leftover pair has no high half
-      int T = pr.len + G * SubLanes<R>::V;         // the last sub-lane finishes column len-1 at step T-2
-      if (G < 32) T = __reduce_max_sync(FULL, T);  // warp-uniform trip count (shuffles)
-      uint32_t best = 0;
-      const bool l2 = q2 || wide;  // query-pair profile geometry
-      const int SBx = l2 ? a.SB2 : a.SB;
-      const int ncp = l2 ? a.ncopy[1] : a.ncopy[0], csx = l2 ? a.cstride[1] : a.cstride[0];
-      const uint32_t skw = l2 ? 0u : a.cskew0;
-      const int rs = d.res_stride;  // > 0: every strip of the slot resident (loaded once per slot)
-      for (int s = 0; s < d.n_strips; ++s) {
-        const int want = rs ? ((sl << 16) | 0xffff) : ((sl << 16) | s);
-        if (want != loaded) {
-          __syncthreads();
-          if (rs) {
-            for (int s2 = 0; s2 < d.n_strips; ++s2)
-              for (int cp = 0; cp < ncp; ++cp)
-                copy_strip(sprof + s2 * rs + copy_off(cp, csx, skw), d.prof + (size_t)s2 * SBx, SBx);
-          } else {
-            for (int cp = 0; cp < ncp; ++cp) copy_strip(sprof + copy_off(cp, csx, skw), d.prof + (size_t)s * SBx, SBx);
-          }
-          __syncthreads();
-          loaded = want;
-        }
-        const uint8_t* gprof = sprof + (rs ? s * rs : 0) + copy_off(g & (ncp - 1), csx, skw);  // this group's bank-spread copy
-        if (q2) {
-          const StripInfo si = d.sinfo[s];
-          const bool rd = s > 0 && si.keep != 0;
-          if (rd && si.keep != FULL) {  // one half starts a new query: zero its half of the boundary row
-            for (int c = k; c < T; c += G) {
-              const uint2 v = bb[c];
-              bb[c] = make_uint2(v.x & si.keep, v.y & si.keep);
-            }
-            __syncwarp();
-          }
-          strip_pass<G, R, false, true>(gprof, a.LS2, a.LB2, a.stream + pr.off, pr.len, T, k, rd,
-                                        s + 1 < d.n_strips, bb, bb, Link{}, a.code_pad2,
-                                        a.nGe, a.nGsGe, best, half ? 8u : 0u);
-          if (si.emit0 >= 0 || si.emit1 >= 0) {  // a query of either half ends with this strip
-            uint32_t bg = best;
-#pragma unroll
-            for (int o = G / 2; o > 0; o >>= 1) bg = __vmaxs2(bg, __shfl_xor_sync(FULL, bg, o, G));
-            if (valid && k == 0) {
-              const int id = half ? pr.id1 : pr.id0;
-              if (si.emit0 >= 0) {
-                const int v = int(int16_t(bg & 0xffffu));
-                a.scores_all[(int64_t)si.emit0 * a.n_seqs + id] = v;
-                if (v >= a.thr) {
-                  const int e = atomicAdd(a.ovf_count, 1);
-                  if (e < a.ovf_cap) a.ovf[e] = OvfRec{si.emit0, p, half, 0};
-                }
-              }
-              if (si.emit1 >= 0) {
-                const int v = int(int16_t(bg >> 16));
-                a.scores_all[(int64_t)si.emit1 * a.n_seqs + id] = v;
-                if (v >= a.thr) {
-                  const int e = atomicAdd(a.ovf_count, 1);
-                  if (e < a.ovf_cap) a.ovf[e] = OvfRec{si.emit1, p, half, 0};
-                }
-              }
-            }
-            best &= (si.emit0 >= 0 ? 0xffff0000u : 0xffffffffu) & (si.emit1 >= 0 ? 0x0000ffffu : 0xffffffffu);
-          }
-        } else {
-          if constexpr (wide)
-            strip_pass<G, R, false, false, 16, 1>(gprof, a.LS2, a.LB2, a.stream + pr.off, pr.len, T, k, s > 0,
-                                                  s + 1 < d.n_strips, bb, bb, Link{}, a.code_pad2, a.nGe, a.nGsGe,
-                                                  best, 0u, a.wmul);
-          else
-            strip_pass<G, R, false>(gprof, a.LS, a.LB, a.stream + pr.off, pr.len, T, k, s > 0, s + 1 < d.n_strips,
-                                    bb, bb, Link{}, a.code_pad2, a.nGe, a.nGsGe, best);
-        }
-      }
-      if (!q2) {  // mode 0: one query, both halves are DB sequences
-#pragma unroll
-        for (int o = G / 2; o > 0; o >>= 1) best = __vmaxs2(best, __shfl_xor_sync(FULL, best, o, G));
-        if (valid && k == 0) {
-          QueryDesc qd;
-          qd.scores = d.scores0;
-          qd.qidx = d.qidx0;
-          emit_pair(a, qd, p, pr, best);
+          wp[t0 + j] = make_uint2(sH, sF);
         }
       }
     }
-    __syncthreads();
+    if constexpr (LINKED) {
+      // progress, every 8 columns: release orders this lane's ring writes before the counter
+      if (wr && tail && (((t0 >> 2) & 1) || t0 + 4 >= T)) st_release_cta(ch.out_prog, ch.out_base + t0 + 4);
+      // consumption: block t0's ring cells were used above (their loads completed), so a
+      // relaxed store suffices -- the producer only overwrites cells below this index
+      if (rd && ch.in_ring && lead && (((t0 >> 2) & 1) || t0 + 4 >= T))
+        st_relaxed_cta(ch.in_cons, ch.in_base + min(t0 + 4 + ioff, T));
+    }
+  }
+  if constexpr (LINKED) {
+    if (rd && ch.in_ring && lead) st_relaxed_cta(ch.in_cons, ch.in_base + T);  // everything consumed
   }
 }
 
-template <int G, int R, int NT>
-#ifdef SW_MINB  // experiments only: __launch_bounds__(NT, 1) lets ptxas take 225 registers (1 CTA/SM, -5% on config 3)
-__global__ void __launch_bounds__(NT, SW_MINB) inter_kernel(InterArgs a) {
-#else
-__global__ void __launch_bounds__(NT) inter_kernel(InterArgs a) {
-#endif
-  inter_body<G, R, NT, 0>(a);
-}
-// the wide-profile variant, held to 2 CTAs/SM (128 registers) like the default
-template <int G, int R, int NT>
-__global__ void __launch_bounds__(NT, 2) inter_kernel_wide(InterArgs a) {
-  inter_body<G, R, NT, 1>(a);
+__device__ __forceinline__ void flag_overflow(int* ovf_count, OvfRec* ovf, int cap, int q, int p, int half) {
+  const int e = atomicAdd(ovf_count, 1);
+  if (e < cap) ovf[e] = OvfRec{q, p, half, 0};
 }
 
 // ---------------------------------------------------------------------------
-// Instantiation table.
-#ifndef SW_INTER_NT
-#define SW_INTER_NT 256
-#endif
-constexpr int INTER_NT = SW_INTER_NT;  // threads per CTA of the scoring kernel
+// Short-pair items: the host ordered all (slot, chunk) items of
+// the launch by critical path (strips x pair length), longest first.
+// Query-pair strip profiles are staged by the TMA engine: two shared-memory
+// buffers, each holding the bank-spread copies of one strip; while the lane groups
+// sweep strip s from one buffer, cp.async.bulk fills the other with strip s+1
+// (completion counted on that buffer's mbarrier).  One CTA barrier per pass.
+struct ProfStage {
+  int tag[2];        // (slot << 16 | strip) held / in flight per buffer, -1: none (CTA-uniform)
+  uint32_t parity;   // bit b: mbarrier phase parity the next wait on buffer b expects
+  uint32_t pending;  // bit b: a bulk copy into buffer b not yet waited for
+  uint64_t* mbar;    // [2] in shared memory
+};
 
-#define SW_INTER_CASES(X)                                                          \
+__device__ __forceinline__ void stage_issue(ProfStage& ps, int b, int tag, const ShortArgs& a, uint8_t* buf,
+                                            const uint8_t* src) {
+  if (threadIdx.x == 0) {
+    fence_proxy_async_smem();  // the buffer's previous strip was read through the generic proxy
+    mbar_arrive_expect_tx(ps.mbar + b, uint32_t(a.ncopy * a.SB));
+    for (int cp = 0; cp < a.ncopy; ++cp) bulk_g2s(buf + cp * a.cstride, src, uint32_t(a.SB), ps.mbar + b);
+  }
+  ps.tag[b] = tag;
+  ps.pending |= 1u << b;
+}
+
+template <int G, int R, int NT, bool Q2>
+__device__ __forceinline__ void short_item(const ShortArgs& a, int item, uint8_t* smem, int& loaded, ProfStage& ps) {
+  uint8_t* sprof = smem;                         // the strip profile (bank-spread copies)
+  constexpr int NG = NT / G;
+  const int tid = threadIdx.x;
+  const int k = tid & (G - 1);
+  const int g = tid / G;
+  // per-group boundary row; offset so that &bb[V*G - 1] is 32-byte aligned (bcap % 4 == 0)
+  constexpr int BB_PAD = (4 - (G * SubLanes<R>::V - 1) % 4) % 4;
+  uint2* __restrict__ bb = a.bbuf + ((size_t)blockIdx.x * NG + g) * (size_t)a.bcap + BB_PAD;
+  {
+    const int2 sc = a.item_map[item];
+    const int sl = sc.x;
+    const SlotDesc d = a.slots[sl];
+    const int chunk = sc.y;
+    int p, half = 0;
+    if constexpr (Q2) {  // chunk of NG half-pairs: DB sequence = one half of a pair
+      const int hp = chunk * NG + g;
+      p = d.pair_begin + (hp >> 1);
+      half = hp & 1;
+    } else {
+      p = d.pair_begin + chunk * NG + g;
+    }
+    bool valid = p < a.pair_end;
+    PairRec pr;
+    if (valid) pr = a.pairs[p];
+    else { pr.off = 0; pr.len = 0; pr.id0 = -1; pr.id1 = -1; }
+    if (Q2 && half && pr.id1 < 0) valid = false;  // odd leftover pair has no high half
+    int T = pr.len + G * SubLanes<R>::V;          // the last sub-lane finishes column len-1 at step T-2
+    if (G < 32) T = __reduce_max_sync(FULL, T);   // warp-uniform trip count (shuffles)
+    uint32_t best = 0;
+    for (int s = 0; s < d.n_strips; ++s) {
+      const int want = (sl << 16) | s;
+      const uint8_t* sbuf = sprof;
+      if constexpr (Q2) {
+        const int bsz = (a.ncopy - 1) * a.cstride + a.SB;
+        const int b = s & 1;
+        __syncthreads();  // every group is done with strip s-1 (the other buffer) and strip s-2 (this one)
+        if (ps.tag[b] != want) stage_issue(ps, b, want, a, sprof + b * ((bsz + 127) & ~127), d.prof + (size_t)s * a.SB);
+        if (s + 1 < d.n_strips && ps.tag[b ^ 1] != want + 1)  // prefetch the next strip
+          stage_issue(ps, b ^ 1, want + 1, a, sprof + (b ^ 1) * ((bsz + 127) & ~127), d.prof + (size_t)(s + 1) * a.SB);
+        if (ps.pending & (1u << b)) {
+          mbar_wait(ps.mbar + b, (ps.parity >> b) & 1u);
+          ps.parity ^= 1u << b;
+          ps.pending &= ~(1u << b);
+        }
+        sbuf = sprof + b * ((bsz + 127) & ~127);
+      } else if (want != loaded) {
+        __syncthreads();
+        for (int cp = 0; cp < a.ncopy; ++cp)
+          copy_strip(sprof + copy_off(cp, a.cstride, a.cskew), d.prof + (size_t)s * a.SB, a.SB);
+        __syncthreads();
+        loaded = want;
+      }
+      const uint8_t* gprof = sbuf + copy_off(g & (a.ncopy - 1), a.cstride, a.cskew);  // this group's copy
+      if constexpr (Q2) {
+        const StripInfo si = d.sinfo[s];
+        const bool rd = s > 0 && si.keep != 0;
+        if (rd && si.keep != FULL) {  // one half starts a new query: zero its half of the boundary row
+          for (int c = k; c < T; c += G) {
+            const uint2 v = bb[c];
+            bb[c] = make_uint2(v.x & si.keep, v.y & si.keep);
+          }
+          __syncwarp();
+        }
+        strip_pass<G, R, false, true>(gprof, a.LS, a.LB, a.stream + pr.off, pr.len, T, k, rd, s + 1 < d.n_strips,
+                                      bb, bb, Chain{}, a.code_pad2, a.nGe, a.nGsGe, best, half ? 8u : 0u);
+        if (si.emit0 >= 0 || si.emit1 >= 0) {  // a query of either half ends with this strip
+          uint32_t bg = best;
+#pragma unroll
+          for (int o = G / 2; o > 0; o >>= 1) bg = __vmaxs2(bg, __shfl_xor_sync(FULL, bg, o, G));
+          if (valid && k == 0) {
+            const int id = half ? pr.id1 : pr.id0;
+            if (si.emit0 >= 0) {
+              const int v = int(int16_t(bg & 0xffffu));
+              a.scores_all[(int64_t)si.emit0 * a.n_seqs + id] = v;
+              if (v >= a.thr) flag_overflow(a.ovf_count, a.ovf, a.ovf_cap, si.emit0, p, half);
+            }
+            if (si.emit1 >= 0) {
+              const int v = int(int16_t(bg >> 16));
+              a.scores_all[(int64_t)si.emit1 * a.n_seqs + id] = v;
+              if (v >= a.thr) flag_overflow(a.ovf_count, a.ovf, a.ovf_cap, si.emit1, p, half);
+            }
+          }
+          best &= (si.emit0 >= 0 ? 0xffff0000u : 0xffffffffu) & (si.emit1 >= 0 ? 0x0000ffffu : 0xffffffffu);
+        }
+      } else {
+        strip_pass<G, R, false>(gprof, a.LS, a.LB, a.stream + pr.off, pr.len, T, k, s > 0, s + 1 < d.n_strips,
+                                bb, bb, Chain{}, a.code_pad2, a.nGe, a.nGsGe, best);
+      }
+    }
+    if constexpr (!Q2) {  // mode 0: one query, both halves are DB sequences
+#pragma unroll
+      for (int o = G / 2; o > 0; o >>= 1) best = __vmaxs2(best, __shfl_xor_sync(FULL, best, o, G));
+      if (valid && k == 0) {
+        const int lo = int(int16_t(best & 0xffffu)), hi = int(int16_t(best >> 16));
+        d.scores0[pr.id0] = lo;
+        if (lo >= a.thr) flag_overflow(a.ovf_count, a.ovf, a.ovf_cap, d.qidx0, p, 0);
+        if (pr.id1 >= 0) {
+          d.scores0[pr.id1] = hi;
+          if (hi >= a.thr) flag_overflow(a.ovf_count, a.ovf, a.ovf_cap, d.qidx0, p, 1);
+        }
+      }
+    }
+  }
+}
+
+// Long-pair items (intra-task mode; the paper's fine-grained
+// wavefront across PEs, Fig. 2): one CTA item = one (query, long pair);
+// its LONG_W warps run the strips of 32 lanes x LONG_R rows round-robin (round r:
+// warp w takes strip LONG_W*r + (LONG_W-1-w); upstream strips on the HIGHER warp
+// ids, which the SMSP arbiter favours, so producers keep their lead).  Strip s
+// consumes strip s-1's bottom row: inside a round through a shared-memory ring
+// (LONG_RING steps; producer progress and consumer progress counters give
+// back-pressure), across the round wrap (the last warp's strip -> the first
+// warp's strip of the next round, which starts only after the first warp's
+// current strip ends) through a global row per CTA.  A pair never spans CTAs:
+// every wait is on a warp of the same CTA, so nothing depends on co-residency.
+struct LongShared {
+  int prog[LONG_W];
+  int cons[LONG_W];
+  uint32_t best[LONG_W];
+};
+
+__device__ __forceinline__ void long_item(const LongArgs& a, int item, uint8_t* smem, LongShared& sh) {
+  constexpr int W = LONG_W;
+  // A producer may run LONG_RING - 4 steps ahead of its consumer's last published
+  // consumption; the consumer starts only once the producer is ioff + 4 +
+  // LINK_LAG steps in, so the ring must hold more than that (else both wait).
+  static_assert(LONG_RING - 4 >= (32 * SubLanes<LONG_R>::V - 1) + 4 + LINK_LAG + 16, "ring too short for the lag");
+  uint2* rings = reinterpret_cast<uint2*>(smem);                       // [W - 1][LONG_RING]
+  uint8_t* lprof = smem + (W - 1) * LONG_RING * sizeof(uint2);         // [W][SBL]
+  int* s_prog = sh.prog;
+  int* s_cons = sh.cons;
+  uint32_t* s_best = sh.best;
+  const int tid = threadIdx.x;
+  const int lane = tid & 31, warp = tid >> 5;
+  uint2* wrap = a.wrap + (size_t)blockIdx.x * a.wcap;
+  {
+    if (tid < W) { s_prog[tid] = -1; s_cons[tid] = 0; s_best[tid] = 0; }
+    __syncthreads();
+    int lo = 0, hi = a.n_queries - 1;
+    while (lo < hi) {
+      const int mid = (lo + hi + 1) >> 1;
+      if (a.queries[mid].item_begin <= item) lo = mid; else hi = mid - 1;
+    }
+    const LongQuery d = a.queries[lo];
+    const int ns = d.n_strips;
+    // a query of fewer strips than warps: P (host-chosen, <= W / ns) pairs per item, ns warps each
+    const int P = d.pack;
+    const int GS = ns >= W ? W : ns;             // warps per pair
+    const int grp = warp / GS, wg = warp - grp * GS;
+    const int j = GS - 1 - wg;                   // position of this warp's strip within a round
+    const int pidx = (item - d.item_begin) * P + grp;
+    const bool active = grp < P && pidx < d.n_long;
+    PairRec pr;
+    if (active) pr = a.pairs[pidx];
+    else { pr.off = 0; pr.len = 0; pr.id0 = -1; pr.id1 = -1; }
+    constexpr int VG = 32 * SubLanes<LONG_R>::V;
+    const int T = pr.len + VG;
+    uint32_t best = 0;
+    uint8_t* myprof = lprof + warp * a.SBL;
+    const int lbase = grp * (GS - 1), cbase = grp * GS;  // this pair's rings and counters
+    for (int r = 0; active; ++r) {
+      const int s = GS * r + j;  // strip index
+      if (s >= ns) break;
+      __syncwarp();
+      {  // this warp's strip profile -> its own slot
+        const uint4* src = reinterpret_cast<const uint4*>(d.prof_long + (size_t)s * a.SBL);
+        uint4* dst = reinterpret_cast<uint4*>(myprof);
+        for (int i = lane; i < a.SBL / 16; i += 32) dst[i] = __ldg(src + i);
+      }
+      __syncwarp();
+      const bool rd = s > 0, wr = s + 1 < ns;
+      Chain ch{};
+      ch.out_base = r * T;
+      // input: ring j-1 (same round) or the wrap row (previous round, from position GS-1)
+      ch.in_ring = j > 0;
+      if (j > 0) {
+        ch.in_sring = static_cast<uint32_t>(__cvta_generic_to_shared(rings + (size_t)(lbase + j - 1) * LONG_RING));
+        ch.in_prog = &s_prog[cbase + j - 1];
+        ch.in_cons = &s_cons[cbase + j - 1];
+        ch.in_base = r * T;
+      } else {
+        ch.in_prog = &s_prog[cbase + GS - 1];
+        ch.grow_in = wrap;
+        ch.in_base = (r - 1) * T;   // the wrap row was written in the previous round
+      }
+      ch.out_ring = j < GS - 1;
+      if (j < GS - 1) {
+        ch.out_sring = static_cast<uint32_t>(__cvta_generic_to_shared(rings + (size_t)(lbase + j) * LONG_RING));
+        ch.out_cons = &s_cons[cbase + j];
+      } else {
+        ch.grow_out = wrap;         // only reached when ns > W (P = 1): the round wrap
+      }
+      ch.out_prog = &s_prog[cbase + j];
+      strip_pass<32, LONG_R, true, false, LONG_US>(myprof, a.LSL, a.LBL, a.stream + pr.off, pr.len, T, lane, rd, wr,
+                                                   nullptr, nullptr, ch, a.code_pad2, a.nGe, a.nGsGe, best);
+    }
+#pragma unroll
+    for (int o = 16; o > 0; o >>= 1) best = __vmaxs2(best, __shfl_xor_sync(FULL, best, o));
+    if (lane == 0) s_best[warp] = best;
+    __syncthreads();
+    if (tid < P) {
+      const int pj = (item - d.item_begin) * P + tid;
+      if (pj < d.n_long) {
+        const PairRec pq = a.pairs[pj];
+        uint32_t b = 0;
+        for (int w = tid * GS; w < tid * GS + GS; ++w) b = __vmaxs2(b, s_best[w]);
+        const int v0 = int(int16_t(b & 0xffffu)), v1 = int(int16_t(b >> 16));
+        d.scores[pq.id0] = v0;
+        if (v0 >= a.thr) flag_overflow(a.ovf_count, a.ovf, a.ovf_cap, d.qidx, pj, 0);
+        if (pq.id1 >= 0) {
+          d.scores[pq.id1] = v1;
+          if (v1 >= a.thr) flag_overflow(a.ovf_count, a.ovf, a.ovf_cap, d.qidx, pj, 1);
+        }
+      }
+    }
+    __syncthreads();
+  }
+}
+// The short-pair kernel: one persistent launch per short-pair mode (query pairs,
+// single query), one (G, R) per launch, its own register budget (the query-pair
+// form keeps R = 32 rows per lane at 128 registers, 2 CTAs per SM).
+template <int G, int R, int NT, bool Q2>
+__global__ void __launch_bounds__(NT, 2) short_kernel(ShortArgs as) {
+  extern __shared__ __align__(128) uint8_t smem[];
+  __shared__ int s_item;
+  __shared__ __align__(8) uint64_t s_mbar[2];
+  int loaded = -1;  // (slot << 16 | strip) of the strip profile in shared memory (CTA-uniform)
+  ProfStage ps{{-1, -1}, 0u, 0u, s_mbar};
+  if (Q2 && threadIdx.x == 0) {
+    mbar_init(s_mbar, 1);
+    mbar_init(s_mbar + 1, 1);
+    asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
+  }
+  for (;;) {
+    if (threadIdx.x == 0) s_item = atomicAdd(as.work_counter, 1);
+    __syncthreads();
+    const int item = s_item;
+    __syncthreads();
+    if (item >= as.n_items) break;
+    short_item<G, R, NT, Q2>(as, item, smem, loaded, ps);
+  }
+}
+
+// A long item as an out-of-line call: the combined single-query kernel below keeps
+// the short path's register allocation apart from it.
+__device__ __noinline__ void long_item_call(const LongArgs& a, int item, uint8_t* smem, LongShared& sh) {
+  long_item(a, item, smem, sh);
+}
+
+// Single-query searches with long pairs (C1/C2): ONE persistent launch, the long
+// items first (costliest), then the short items, so the longest pairs start at
+// once and the SMs that finish them move on to short items.
+template <int G, int R, int NT>
+__global__ void __launch_bounds__(NT, 2) combined_m0_kernel(ShortArgs as, LongArgs al) {
+  extern __shared__ __align__(128) uint8_t smem[];
+  __shared__ int s_item;
+  __shared__ LongShared sh;
+  int loaded = -1;
+  ProfStage ps{{-1, -1}, 0u, 0u, nullptr};  // (single-query items copy their profile by hand)
+  const int n_items = al.n_items + as.n_items;
+  for (;;) {
+    if (threadIdx.x == 0) s_item = atomicAdd(as.work_counter, 1);
+    __syncthreads();
+    const int item = s_item;
+    __syncthreads();
+    if (item >= n_items) break;
+    if (item < al.n_items) {
+      long_item_call(al, item, smem, sh);
+      loaded = -1;  // the long item overwrote the strip profile
+    } else {
+      short_item<G, R, NT, false>(as, item - al.n_items, smem, loaded, ps);
+    }
+  }
+}
+
+// The long-pair (intra-task) kernel: one persistent launch, costliest items first.
+// When short pairs are scored too it runs concurrently with the short-pair kernel
+// on a side stream, one CTA per SM (a shared-memory request that leaves no room
+// for a short-pair CTA), so the co-resident short warps do not stretch the
+// critical path of the longest pairs.
+__global__ void __launch_bounds__(LONG_W * 32, 2) long_kernel(LongArgs al) {
+  extern __shared__ __align__(128) uint8_t smem[];
+  __shared__ int s_item;
+  __shared__ LongShared sh;
+  for (;;) {
+    if (threadIdx.x == 0) s_item = atomicAdd(al.work_counter, 1);
+    __syncthreads();
+    const int item = s_item;
+    __syncthreads();
+    if (item >= al.n_items) break;
+    long_item(al, item, smem, sh);
+  }
+}
+
+// ---------------------------------------------------------------------------
+// Instantiation tables.
+typedef void (*short_fn)(ShortArgs);
+#define SW_GEOM_CASES(X)                                                           \
   X(4, 8) X(4, 12) X(4, 16) X(4, 20) X(4, 24) X(4, 28) X(4, 32)                    \
   X(8, 8) X(8, 12) X(8, 16) X(8, 20) X(8, 24) X(8, 28) X(8, 32)                    \
   X(16, 8) X(16, 12) X(16, 16) X(16, 20) X(16, 24) X(16, 28) X(16, 32)             \
   X(32, 8) X(32, 12) X(32, 16) X(32, 20) X(32, 24) X(32, 28) X(32, 32)
 
-typedef void (*inter_fn)(InterArgs);
-
-#define SW_WIDE_CASES(X) X(4, 24) X(8, 24) X(8, 16) X(16, 24) X(8, 32) X(4, 16)
-
-static inter_fn pick_inter(int G, int R, int NT, int wide = 0) {
-  if (NT != INTER_NT) return nullptr;
-  if (wide) {
-#define X(g, r) \
-    if (G == g && R == r) return inter_kernel_wide<g, r, INTER_NT>;
-    SW_WIDE_CASES(X)
+static short_fn pick_short(int mode, int G, int R) {
+  if (mode == 1) {
+#define X(g, r) if (G == g && R == r) return short_kernel<g, r, SCORE_NT, true>;
+    SW_GEOM_CASES(X)
 #undef X
-    return nullptr;
+  } else {
+#define X(g, r) if (G == g && R == r) return short_kernel<g, r, SCORE_NT, false>;
+    SW_GEOM_CASES(X)
+#undef X
   }
-#define X(g, r) \
-  if (G == g && R == r) return inter_kernel<g, r, INTER_NT>;
-  SW_INTER_CASES(X)
-#undef X
   return nullptr;
 }
 
-bool inter_config_supported(int G, int R) { return pick_inter(G, R, INTER_NT) != nullptr; }
-bool inter_wide_supported(int G, int R) { return pick_inter(G, R, INTER_NT, 1) != nullptr; }
-int inter_block_threads() { return INTER_NT; }
+bool short_config_supported(int mode, int G, int R) { return pick_short(mode, G, R) != nullptr; }
 
-int inter_max_ctas_per_sm(int G, int R, int NT, int smem_bytes, int wide) {
-  inter_fn f = pick_inter(G, R, NT, wide);
-  if (!f) return 0;
-  if (smem_bytes > 48 * 1024)
-    cudaFuncSetAttribute(f, cudaFuncAttributeMaxDynamicSharedMemorySize, smem_bytes);
+static int occupancy(const void* f, int threads, int smem_bytes) {
+  if (smem_bytes > 48 * 1024) cudaFuncSetAttribute(f, cudaFuncAttributeMaxDynamicSharedMemorySize, smem_bytes);
   int n = 0;
-  if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&n, f, NT, smem_bytes) != cudaSuccess) return 0;
+  if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&n, f, threads, smem_bytes) != cudaSuccess) return 0;
   return n;
 }
 
-cudaError_t launch_inter(int G, int R, int NT, int grid, int smem_bytes, const InterArgs& a, cudaStream_t st,
-                         int wide) {
-  inter_fn f = pick_inter(G, R, NT, wide);
+int short_max_ctas_per_sm(int mode, int G, int R, int smem_bytes) {
+  short_fn f = pick_short(mode, G, R);
+  return f ? occupancy(reinterpret_cast<const void*>(f), SCORE_NT, smem_bytes) : 0;
+}
+
+cudaError_t launch_short(int mode, int G, int R, int grid, int smem_bytes, const ShortArgs& a, cudaStream_t st) {
+  short_fn f = pick_short(mode, G, R);
   if (!f) return cudaErrorInvalidValue;
   if (smem_bytes > 48 * 1024) {
     cudaError_t e = cudaFuncSetAttribute(f, cudaFuncAttributeMaxDynamicSharedMemorySize, smem_bytes);
     if (e != cudaSuccess) return e;
   }
-  f<<<grid, NT, smem_bytes, st>>>(a);
+  f<<<grid, SCORE_NT, smem_bytes, st>>>(a);
+  return cudaGetLastError();
+}
+
+typedef void (*combined_fn)(ShortArgs, LongArgs);
+static combined_fn pick_combined(int G, int R) {
+#define X(g, r) if (G == g && R == r) return combined_m0_kernel<g, r, SCORE_NT>;
+  SW_GEOM_CASES(X)
+#undef X
+  return nullptr;
+}
+
+int combined_max_ctas_per_sm(int G, int R, int smem_bytes) {
+  combined_fn f = pick_combined(G, R);
+  return f ? occupancy(reinterpret_cast<const void*>(f), SCORE_NT, smem_bytes) : 0;
+}
+
+cudaError_t launch_combined(int G, int R, int grid, int smem_bytes, const ShortArgs& as, const LongArgs& al,
+                            cudaStream_t st) {
+  combined_fn f = pick_combined(G, R);
+  if (!f) return cudaErrorInvalidValue;
+  if (smem_bytes > 48 * 1024) {
+    cudaError_t e = cudaFuncSetAttribute(f, cudaFuncAttributeMaxDynamicSharedMemorySize, smem_bytes);
+    if (e != cudaSuccess) return e;
+  }
+  f<<<grid, SCORE_NT, smem_bytes, st>>>(as, al);
+  return cudaGetLastError();
+}
+
+int long_max_ctas_per_sm(int smem_bytes) {
+  return occupancy(reinterpret_cast<const void*>(long_kernel), LONG_W * 32, smem_bytes);
+}
+
+cudaError_t launch_long(int grid, int smem_bytes, const LongArgs& a, cudaStream_t st) {
+  if (smem_bytes > 48 * 1024) {
+    cudaError_t e = cudaFuncSetAttribute(long_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize, smem_bytes);
+    if (e != cudaSuccess) return e;
+  }
+  long_kernel<<<grid, LONG_W * 32, smem_bytes, st>>>(a);
   return cudaGetLastError();
 }
 
@@ -801,7 +808,7 @@ __global__ void __launch_bounds__(RESCORE_WARPS * 32) rescore_kernel(RescoreArgs
     int2* grow = a.grows + (int64_t)blk * K * a.bcap;
     unsigned long long* gflag = a.gflags + (int64_t)blk * K;
     const unsigned long long gen = (unsigned long long)(e + 1) << 32;
-    const int j = W - 1 - warp;  // producers on higher warp ids (see inter_kernel)
+    const int j = W - 1 - warp;  // producers on higher warp ids (see long_kernel)
     const int s = W * c + j;
     // the block's previous entry must be finished before this CTA writes its row
     if (c + 1 < K && e >= a.ne_slots && warp == 0) {

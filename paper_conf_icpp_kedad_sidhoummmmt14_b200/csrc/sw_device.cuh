@@ -44,24 +44,6 @@ __host__ __device__ constexpr int lane_block_bytes(int R) {
   return ((R % 8 == 0) ? (((R / 8) | 1) * 8) : (((R / 4) | 1) * 4));
 }
 
-// Boundary rows of multi-strip lane groups are rewritten and re-read once per
-// strip pass: keep them in L2 (evict_last) while the DB codes stream through
-// with evict-first loads, so they need not travel to DRAM and back.
-__device__ __forceinline__ uint64_t l2_evict_last_policy() {
-  uint64_t p;
-  asm volatile("createpolicy.fractional.L2::evict_last.b64 %0, 1.0;" : "=l"(p));
-  return p;
-}
-__device__ __forceinline__ uint4 ld_l2_last(const void* a, uint64_t pol) {
-  uint4 v;
-  asm volatile("ld.global.L2::cache_hint.v4.u32 {%0, %1, %2, %3}, [%4], %5;"
-               : "=r"(v.x), "=r"(v.y), "=r"(v.z), "=r"(v.w) : "l"(a), "l"(pol));
-  return v;
-}
-__device__ __forceinline__ void st_l2_last(void* a, uint2 v, uint64_t pol) {
-  asm volatile("st.global.L2::cache_hint.v2.u32 [%0], {%1, %2}, %3;" :: "l"(a), "r"(v.x), "r"(v.y), "l"(pol) : "memory");
-}
-
 // Shared-memory loads by 32-bit shared-window address (the profile pointers
 // stay 32-bit: fewer registers than generic 64-bit pointers, no address
 // rematerialisation in the hot loop).
@@ -149,28 +131,14 @@ __device__ __forceinline__ void gotoh_rows_inplace(uint32_t (&H)[R], uint32_t (&
 }
 
 // Profile values S(q_r, letter) of rows [R0, R1) for one lane (see gotoh_rows_inplace).
-// PW (wide single-query profile): 32-bit rows holding S & 0xffff; the pair
-// (S[b] : S[a]) is one IMAD, S[b] * 2^16 + S[a], on the FMA pipe instead of a
-// PRMT on the ALU pipe (wmul = 65536, a runtime value so that it stays an IMAD).
-__device__ __forceinline__ uint32_t imad_u32(uint32_t a, uint32_t b, uint32_t c) {
-  uint32_t d;
-  asm("mad.lo.u32 %0, %1, %2, %3;" : "=r"(d) : "r"(a), "r"(b), "r"(c));
-  return d;
-}
-
-template <int R, int R0, int R1, bool Q2, int US, int PW = 0>
-__device__ __forceinline__ void load_rows(uint32_t (&sv)[R1 - R0], uint32_t pa, uint32_t pb, uint32_t wmul = 0) {
+template <int R, int R0, int R1, bool Q2, int US>
+__device__ __forceinline__ void load_rows(uint32_t (&sv)[R1 - R0], uint32_t pa, uint32_t pb) {
   constexpr int N = R1 - R0;
-  constexpr int UB = (Q2 || PW) ? 4 : ((R % 8 == 0 && R0 % 8 == 0 && N % 8 == 0) ? 8 : 4);
+  constexpr int UB = Q2 ? 4 : ((R % 8 == 0 && R0 % 8 == 0 && N % 8 == 0) ? 8 : 4);
 #pragma unroll
   for (int u = R0 / UB; u < R1 / UB; ++u) {
     const int b = u * UB - R0;
-    if constexpr (PW) {
-      const uint4 x = lds128(pa + u * US);
-      const uint4 y = lds128(pb + u * US);
-      sv[b] = imad_u32(y.x, wmul, x.x); sv[b + 1] = imad_u32(y.y, wmul, x.y);
-      sv[b + 2] = imad_u32(y.z, wmul, x.z); sv[b + 3] = imad_u32(y.w, wmul, x.w);
-    } else if constexpr (Q2) {
+    if constexpr (Q2) {
       const uint4 w = lds128(pa + u * US);
       sv[b] = w.x; sv[b + 1] = w.y; sv[b + 2] = w.z; sv[b + 3] = w.w;
     } else if constexpr (UB == 8) {
@@ -194,17 +162,16 @@ __device__ __forceinline__ void load_rows(uint32_t (&sv)[R1 - R0], uint32_t pa, 
 // Hio1 / Fio1 are sub-lane 0's outputs of the previous step).  The two F
 // chains are independent, so emitting their rows alternately hands the
 // scheduler two ready instructions per dependency step.
-template <int R, bool Q2, int US, int PW = 0>
+template <int R, bool Q2, int US>
 __device__ __forceinline__ void gotoh_rows_dual(uint32_t (&H)[R], uint32_t (&E)[R], uint32_t& best,
                                                 uint32_t& hdiag0, uint32_t pa0, uint32_t pb0, uint32_t& Hio0,
                                                 uint32_t& Fio0, uint32_t& hdiag1, uint32_t pa1, uint32_t pb1,
-                                                uint32_t& Hio1, uint32_t& Fio1, uint32_t nGe, uint32_t nGsGe,
-                                                uint32_t wmul = 0) {
+                                                uint32_t& Hio1, uint32_t& Fio1, uint32_t nGe, uint32_t nGsGe) {
   constexpr int RH = R / 2;
   static_assert(R % 8 == 0, "two sub-lanes of whole 4-row units");
   uint32_t s0[RH], s1[RH];
-  load_rows<R, 0, RH, Q2, US, PW>(s0, pa0, pb0, wmul);
-  load_rows<R, RH, R, Q2, US, PW>(s1, pa1, pb1, wmul);
+  load_rows<R, 0, RH, Q2, US>(s0, pa0, pb0);
+  load_rows<R, RH, R, Q2, US>(s1, pa1, pb1);
   uint32_t F0 = Fio0, F1 = Fio1;
   uint32_t d0 = __vadd2(hdiag0, s0[0]);
   uint32_t d1 = __vadd2(hdiag1, s1[0]);
@@ -244,19 +211,49 @@ __host__ __device__ constexpr int lane_block_bytes_q2(int R) { return (((R / 4) 
 
 constexpr uint32_t FULL = 0xffffffffu;
 
-// Progress counters of chained strips.  Within a CTA they live in shared memory
-// (CTA-scope release/acquire); between the CTAs that hold consecutive
-// "superstrips" of one long pair they live in global memory (GPU scope).
+// Progress counters of chained strips (shared memory, CTA-scope release/acquire).
 __device__ __forceinline__ int ld_acquire_cta(const int* p) {
   int v;
   asm volatile("ld.acquire.cta.shared.b32 %0, [%1];"
                : "=r"(v) : "r"(static_cast<uint32_t>(__cvta_generic_to_shared(const_cast<int*>(p)))) : "memory");
   return v;
 }
+__device__ __forceinline__ void st_relaxed_cta(int* p, int v) {
+  asm volatile("st.relaxed.cta.shared.b32 [%0], %1;"
+               :: "r"(static_cast<uint32_t>(__cvta_generic_to_shared(p))), "r"(v) : "memory");
+}
 __device__ __forceinline__ void st_release_cta(int* p, int v) {
   asm volatile("st.release.cta.shared.b32 [%0], %1;"
                :: "r"(static_cast<uint32_t>(__cvta_generic_to_shared(p))), "r"(v) : "memory");
 }
+
+// ---------------------------------------------------------------------------
+// Bulk asynchronous copies (TMA engine, cp.async.bulk) global -> shared memory,
+// completion counted in bytes on an mbarrier.
+__device__ __forceinline__ uint32_t smem_u32(const void* p) {
+  return static_cast<uint32_t>(__cvta_generic_to_shared(p));
+}
+__device__ __forceinline__ void mbar_init(uint64_t* m, uint32_t count) {
+  asm volatile("mbarrier.init.shared::cta.b64 [%0], %1;" :: "r"(smem_u32(m)), "r"(count) : "memory");
+}
+__device__ __forceinline__ void mbar_arrive_expect_tx(uint64_t* m, uint32_t bytes) {
+  asm volatile("mbarrier.arrive.expect_tx.shared::cta.b64 _, [%0], %1;" :: "r"(smem_u32(m)), "r"(bytes) : "memory");
+}
+__device__ __forceinline__ void bulk_g2s(void* dst, const void* src, uint32_t bytes, uint64_t* m) {
+  asm volatile("cp.async.bulk.shared::cluster.global.mbarrier::complete_tx::bytes [%0], [%1], %2, [%3];"
+               :: "r"(smem_u32(dst)), "l"(src), "r"(bytes), "r"(smem_u32(m)) : "memory");
+}
+__device__ __forceinline__ void mbar_wait(uint64_t* m, uint32_t parity) {
+  asm volatile("{\n .reg .pred p;\n"
+               "WAIT_%=:\n mbarrier.try_wait.parity.shared::cta.b64 p, [%0], %1;\n"
+               " @!p bra WAIT_%=;\n}" :: "r"(smem_u32(m)), "r"(parity) : "memory");
+}
+// generic-proxy accesses of shared memory before async-proxy (bulk copy) writes
+__device__ __forceinline__ void fence_proxy_async_smem() {
+  asm volatile("fence.proxy.async.shared::cta;" ::: "memory");
+}
+
+// GPU-scope counters (sw_align's CTA-to-CTA chains of very tall pairs).
 __device__ __forceinline__ int ld_acquire_gpu(const int* p) {
   int v;
   asm volatile("ld.acquire.gpu.global.b32 %0, [%1];" : "=r"(v) : "l"(p) : "memory");
@@ -266,8 +263,8 @@ __device__ __forceinline__ void st_release_gpu(int* p, int v) {
   asm volatile("st.release.gpu.global.b32 [%0], %1;" :: "l"(p), "r"(v) : "memory");
 }
 
-// Link of a chained strip: the row above (read by lane 0) and this strip's
-// bottom row (written by the last lane), each with a progress counter.
+// Link of a chained strip (sw_align): the row above (read by lane 0) and this
+// strip's bottom row (written by the last lane), each with a progress counter.
 struct Link {
   int* in;        // counter of the producer of the row above (nullptr: none)
   int in_base;    // value the producer publishes before its first cell

@@ -50,37 +50,43 @@ struct ProfGeom {
   int il;          // 1: unit-interleaved [letter][unit][lane][UB] (long mode); 0: [letter][lane][LB]
 };
 
-#ifndef SW_LONG_R
-#define SW_LONG_R 16
-#endif
-constexpr int LONG_R = SW_LONG_R;   // rows per lane of the intra-task (long pair) geometry, G = 32;
-                             // profile unit-interleaved ([letter][unit][lane][8 B]): dense and
-                             // bank-conflict-free (the 16 lanes of an LDS.64 phase hit 16 distinct
-                             // 8-byte slots whatever letters they read)
-#ifndef SW_LONG_IL
-#define SW_LONG_IL 1
-#endif
-#ifndef SW_SMEM_UNION
-#define SW_SMEM_UNION 1
-#endif
-constexpr int LONG_US = SW_LONG_IL ? 32 * 8 : 8;  // bytes between a lane's consecutive 8-byte units in the long profile
+// Rows per lane of the intra-task (long pair) geometry, G = 32 lanes; profile
+// unit-interleaved ([letter][unit][lane][8 B]): dense and bank-conflict-free (the
+// 16 lanes of an LDS.64 phase hit 16 distinct 8-byte slots whatever letters they read)
+constexpr int LONG_R = 16;
+constexpr int LONG_US = 32 * 8;     // bytes between a lane's consecutive 8-byte units in the long profile
+constexpr int LONG_RING = 128;      // steps held by a shared-memory link ring between two warps of a CTA
 
-// Per-query descriptor of a multi-query launch (processing order: longest first).
-struct QueryDesc {
-  const uint8_t* prof;       // short-pair (inter-task) profile, [n_strips][SB]
-  const uint8_t* prof_long;  // long-pair (intra-task) profile, [n_strips_long][SBL]
+// Long (intra-task) work of one query: pairs [0, n_long) of the DB are scored by
+// the chained warps of one CTA each.
+struct LongQuery {
+  const uint8_t* prof_long;  // [n_strips][SBL] int8, 32 lanes x LONG_R rows per strip
   int32_t* scores;           // this query's row of scores[Q][N] (caller order)
-  int n_strips, n_strips_long;
+  int n_strips;
   int qidx;
-  int n_super;               // superstrips of W = NT/32 strips per long pair
-  int long_item_begin;       // first long work item of this query (n_long * n_super items)
-  int flag_base;             // this query's superstrip counters: gflags[flag_base + pair * n_super + k]
-  int done_base;             // per-pair superstrip completion counters: gdone[done_base + pair]
-  int n_long;                // pairs [0, n_long) are this query's long items
-  int pairs_per_item;        // > 1: the query has fewer than W strips; a long item holds W/strips pairs
-  int pad2_;
-  int64_t glink_base;        // boundary rows: glinks[glink_base + c * glink_stride + lofs[pair] ...]
-  int64_t glink_stride;      // sum over this query's long pairs of (len + 72)
+  int item_begin;            // first long item of this query
+  int n_long;
+  int pack;                  // pairs per item: 1, or up to W / n_strips when n_strips < W (the
+                             // CTA's warps then chain several pairs side by side)
+  int pad_;
+};
+
+struct LongArgs {
+  const LongQuery* queries;  // [n_queries], processing order
+  int n_queries;
+  int n_items;               // sum of n_long
+  int SBL, LSL, LBL;         // long profile geometry
+  uint2* wrap;               // [gridDim][wcap]: the round-wrap link row of each CTA (warp W-1 -> warp 0)
+  int wcap;
+  const uint16_t* stream;
+  const PairRec* pairs;
+  int* work_counter;
+  int32_t thr;               // overflow threshold (int16 max >= thr -> re-score)
+  OvfRec* ovf;
+  int* ovf_count;
+  int ovf_cap;
+  uint32_t code_pad2;        // PAD | PAD << 8
+  uint32_t nGe, nGsGe;       // packed s16x2 -Ge, -(Gs+Ge)
 };
 
 // Short-pair work of one "slot": a single query (mode 0: two DB sequences per
@@ -98,60 +104,42 @@ struct StripInfo {
 
 struct SlotDesc {
   const StripInfo* sinfo;    // mode 1: [n_strips]
-  const uint8_t* prof;       // mode 0: [n_strips][SB] int8; mode 1: [n_strips][SB2] s16x2
-  int32_t* scores0;          // scores row of the (first) query
-  int32_t* scores1;          // mode 1: row of the second query
+  const uint8_t* prof;       // mode 0: [n_strips][SB] int8; mode 1: [n_strips][SB] s16x2
+  int32_t* scores0;          // mode 0: the query's scores row
   int n_strips;
   int mode;
-  int qidx0, qidx1;
-  int item_begin;            // first short work item of this slot
+  int qidx0;
   int n_items;               // short work items of this slot
   int pair_begin;            // short pairs of this slot: [pair_begin, pair_end)
-  int res_stride;            // > 0: all strips resident in smem, strip s at s * res_stride (bytes)
-  int wide;                  // mode 0 with the 32-bit profile (S & 0xffff per row, query-pair geometry)
   int pad_;
 };
 
-struct InterArgs {
-  const QueryDesc* queries;  // [n_queries], processing order (long items)
-  int n_queries;
-  const SlotDesc* slots;     // [n_slots] short-pair work
+// One short-pair kernel launch (all slots of one mode).
+struct ShortArgs {
+  const SlotDesc* slots;
   int n_slots;
-  int n_short_items;         // sum of slots' n_items
-  const int2* item_map;      // short item -> (slot, chunk), longest critical path first
-  int SB, LS, LB;            // short geometry (G, R of the launch), mode 0 profile
-  int SB2, LS2, LB2;         // mode 1 (query-pair) profile
-  // Bank-spread copies of the short strip profile in shared memory: lane group g
-  // reads copy g % ncopy at byte offset (g % ncopy) * cstride; cstride is
-  // 128/ncopy modulo 128, so the groups of one shared-memory phase (random
-  // letters each) hit disjoint banks.  Index 0: mode 0, index 1: mode 1.
-  int ncopy[2], cstride[2];
-  // per-copy bank skew of the mode-0 copies: copy c sits at c * cstride[0] +
-  // 4 * ((cskew0 >> 8c) & 0xff) (0 for the linear layout; mode 1 is always linear)
-  uint32_t cskew0;
-  uint32_t wmul;             // 65536 (runtime, so the wide mode's pair build stays an IMAD)
-  int SBL, LSL, LBL;         // long geometry (32 lanes x LONG_R rows)
-  int n_long_items;          // sum over queries of n_long * n_super
-  uint2* links;              // [gridDim][NT/32][lcap] strip-to-strip rows inside a CTA (long items)
-  int lcap;
-  uint2* glinks;             // superstrip boundary rows (between CTAs)
-  int* gflags;               // their progress counters (zeroed per search)
-  int* gdone;                // per (query, long pair) superstrip completion counters (zeroed per search)
-  const int64_t* lofs;       // per pair: offset of its boundary row (sum of (len + 72) before it)
+  int n_items;
+  const int2* item_map;      // item -> (slot, chunk), longest critical path first
+  int SB, LS, LB;            // strip profile geometry of this mode
+  // Bank-spread copies of the strip profile in shared memory: lane group g reads
+  // copy g % ncopy at ncopy-dependent offsets (copy_off), so the groups of one
+  // shared-memory phase (random letters each) hit disjoint banks.
+  int ncopy, cstride;
+  uint32_t cskew;            // per-copy 4-byte skews (mode 0), 0 for the linear layout
   const uint16_t* stream;
   const PairRec* pairs;
-  int pair_end;              // number of pairs
-  uint2* bbuf;               // boundary rows of multi-strip short items, [gridDim][NG][bcap]
+  int pair_end;
+  uint2* bbuf;               // boundary rows of multi-strip items, [gridDim][NG][bcap]
   int bcap;
   int* work_counter;
-  int32_t* scores_all;       // [n_queries (caller order)][n_seqs]: mode-1 emission target
+  int32_t* scores_all;       // [n_queries (caller order)][n_seqs]
   int64_t n_seqs;
-  int32_t thr;               // overflow threshold (int16 max >= thr -> re-score)
+  int32_t thr;
   OvfRec* ovf;
   int* ovf_count;
   int ovf_cap;
-  uint32_t code_pad2;        // PAD | PAD << 8
-  uint32_t nGe, nGsGe;       // packed s16x2 -Ge, -(Gs+Ge)
+  uint32_t code_pad2;
+  uint32_t nGe, nGsGe;
 };
 
 struct RescoreArgs {
@@ -193,12 +181,19 @@ cudaError_t launch_build_profile(const uint8_t* q, int m, const int8_t* matrix, 
 cudaError_t launch_build_profile_q2(const uint8_t* qa, int ma, const uint8_t* qb, int mb, const int8_t* matrix,
                                     int alpha, int G, int R, int LB2, int LS2, int n_strips, int SB2, uint8_t* prof,
                                     cudaStream_t st);
-int inter_max_ctas_per_sm(int G, int R, int NT, int smem_bytes, int wide = 0);
-cudaError_t launch_inter(int G, int R, int NT, int grid, int smem_bytes, const InterArgs& a, cudaStream_t st,
-                         int wide = 0);
-bool inter_wide_supported(int G, int R);
-bool inter_config_supported(int G, int R);
-int inter_block_threads();  // NT of the scoring kernel (its long items use NT/32 chained warps)
+// Short-pair kernels: mode 0 (single query) and mode 1 (query pairs), one (G, R)
+// per launch.  Long-pair kernel: LONG_W chained warps per CTA.
+constexpr int SCORE_NT = 256;       // threads per CTA of both
+constexpr int LONG_W = SCORE_NT / 32;
+bool short_config_supported(int mode, int G, int R);
+int short_max_ctas_per_sm(int mode, int G, int R, int smem_bytes);
+cudaError_t launch_short(int mode, int G, int R, int grid, int smem_bytes, const ShortArgs& a, cudaStream_t st);
+int long_max_ctas_per_sm(int smem_bytes);
+// single-query searches with long pairs: long items and mode-0 short items in one launch
+int combined_max_ctas_per_sm(int G, int R, int smem_bytes);
+cudaError_t launch_combined(int G, int R, int grid, int smem_bytes, const ShortArgs& as, const LongArgs& al,
+                            cudaStream_t st);
+cudaError_t launch_long(int grid, int smem_bytes, const LongArgs& a, cudaStream_t st);
 cudaError_t launch_rescore(int grid, const RescoreArgs& a, cudaStream_t st);
 // scores[q * stride + cols[c]] = 0 for every query q < nq and column c < ncols
 cudaError_t launch_zero_columns(int32_t* scores, int64_t stride, int nq, const int64_t* cols, int64_t ncols,

@@ -204,19 +204,6 @@ def test_intra_task_mode_forced():
     np.testing.assert_array_equal(got, oracle_scores(qc, qo, dc, do))
 
 
-def test_intra_task_packed_long_pairs():
-    """Option pack_long: a query with fewer intra-task strips than warps scores
-    W / S long pairs per CTA item (S warps per pair); odd pair counts leave a
-    partly filled last item."""
-    rng = np.random.default_rng(23)
-    dl = list(rng.integers(1, 900, size=75)) + [0, 1, 65, 66, 67]
-    dc, do = _seqs(dl, rng)
-    ql = [1, 100, 511, 512, 513, 1500, 2100, 4100]   # 1, 1, 1, 1, 2, 3, 5, 9 strips of 512 rows
-    qc, qo = _seqs(ql, rng)
-    got = gpu_scores(qc, qo, dc, do, opts={"t_long": 64, "pack_long": 1})
-    np.testing.assert_array_equal(got, oracle_scores(qc, qo, dc, do))
-
-
 @pytest.mark.parametrize("pairs", [0, 1])
 @pytest.mark.parametrize("G,R", [(4, 24), (8, 24), (16, 12)])
 def test_profile_without_bank_copies(G, R, pairs):
@@ -287,19 +274,6 @@ def test_query_packing(pack, thr):
     np.testing.assert_array_equal(got, oracle_scores(qc, qo, dc, do))
 
 
-@pytest.mark.parametrize("G,R", [(8, 24), (4, 24), (8, 16), (16, 24), (8, 32), (4, 16)])
-def test_wide_single_query_profile(G, R):
-    """Single-query mode with the wide profile (option wide_profile: 32-bit rows,
-    the (S[b] : S[a]) pair built by one IMAD instead of a PRMT; its own kernel
-    instantiation); multi-strip queries, ragged DB, PAD columns."""
-    rng = np.random.default_rng(81 + G + R)
-    dc, do = _seqs(list(rng.integers(1, 350, size=120)) + [0, 1, 3], rng, alpha=24)
-    qc, qo = _seqs([3 * G * R + 7, G * R, 17, 1], rng, alpha=24)
-    opts = {"wide_profile": 1, "query_pairs": 0, "force_G": G, "force_R": R}
-    got = gpu_scores(qc, qo, dc, do, opts=opts)
-    np.testing.assert_array_equal(got, oracle_scores(qc, qo, dc, do))
-
-
 @pytest.mark.parametrize("skew", [0, 1])
 @pytest.mark.parametrize("G,R", [(8, 24), (8, 8), (16, 24), (16, 8), (8, 12), (4, 16), (8, 16)])
 def test_single_query_profile_copies(G, R, skew):
@@ -310,21 +284,6 @@ def test_single_query_profile_copies(G, R, skew):
     dc, do = _seqs(list(rng.integers(1, 350, size=120)) + [0, 1, 3], rng)
     qc, qo = _seqs([3 * G * R + 7, G * R, 17], rng)
     opts = {"bank_skew": skew, "query_pairs": 0, "force_G": G, "force_R": R}
-    got = gpu_scores(qc, qo, dc, do, opts=opts)
-    np.testing.assert_array_equal(got, oracle_scores(qc, qo, dc, do))
-
-
-@pytest.mark.parametrize("resident", [0, 1])
-@pytest.mark.parametrize("pairs", [0, 1])
-def test_resident_strip_profiles(resident, pairs):
-    """Multi-strip slots whose whole profile fits in shared memory keep every
-    strip resident (loaded once per slot); taller ones stream a strip per pass.
-    One search mixes both (2..6-strip queries and a 190-strip one at 32-row
-    strips), in the query-pair and single-query modes."""
-    rng = np.random.default_rng(61 + 2 * resident + pairs)
-    dc, do = _seqs(list(rng.integers(1, 400, size=140)) + [0, 1, 2, 5], rng)
-    qc, qo = _seqs([6077, 150, 64, 65, 33, 190, 31], rng)
-    opts = {"resident_strips": resident, "query_pairs": pairs, "force_G": 4, "force_R": 8}
     got = gpu_scores(qc, qo, dc, do, opts=opts)
     np.testing.assert_array_equal(got, oracle_scores(qc, qo, dc, do))
 

@@ -31,8 +31,8 @@ template <int R, int NCH, int LDS, int XCH>
 __global__ void k_cell(uint32_t* out, uint32_t seed, int cols) {
   constexpr int RC = R / NCH;
   static_assert(!LDS || RC % 4 == 0, "4-row units");
-  __shared__ __align__(16) uint32_t prof[20 * 8 * (R + 4)];  // [letter][lane % 8][row] (padded lane block)
-  for (int i = threadIdx.x; i < 20 * 8 * (R + 4); i += blockDim.x) prof[i] = (i * 2654435761u) & 0x00070007u;
+  __shared__ __align__(16) uint32_t prof[16 * 8 * (R + 4)];  // [letter][lane % 8][row] (padded lane block)
+  for (int i = threadIdx.x; i < 16 * 8 * (R + 4); i += blockDim.x) prof[i] = (i * 2654435761u) & 0x00070007u;
   __syncthreads();
   const uint32_t sbase = static_cast<uint32_t>(__cvta_generic_to_shared(prof));
   const int lane = threadIdx.x & 31;
@@ -53,14 +53,14 @@ __global__ void k_cell(uint32_t* out, uint32_t seed, int cols) {
       const bool lead = (lane & 3) == 0;
       rH = lead ? hin : rH;
       rF = lead ? fin : rF;
-      rC = lead ? ((t * 7 + 3) % 24) : rC;
+      rC = lead ? ((t * 7 + 3) & 15) : rC;
       hin = rH ^ t;
       fin = rF;
       code = rC;
       F[0] = rF & 0x7fff7fffu;
       hd[0] = rH & 0x7fff7fffu;
     } else {
-      code = (code * 5 + 1) % 24;
+      code = (code * 5 + 1) & 15;
     }
 #pragma unroll
     for (int c = 0; c < NCH; ++c) {
@@ -70,7 +70,7 @@ __global__ void k_cell(uint32_t* out, uint32_t seed, int cols) {
         const int r = c * RC + i;
         if constexpr (LDS) {
           if (i % 4 == 0) {
-            const uint4 w = lds128(sbase + ((code + c) % 20) * 8 * (R + 4) * 4 + laneoff + i * 4);
+            const uint4 w = lds128(sbase + ((code + c) & 15) * (8 * (R + 4) * 4) + laneoff + i * 4);
             S[r] = w.x; S[r + 1] = w.y; S[r + 2] = w.z; S[r + 3] = w.w;
           }
         }
@@ -132,30 +132,24 @@ int main() {
   cudaDeviceProp p; CK(cudaGetDeviceProperties(&p, 0));
   const int sms = p.multiProcessorCount;
   uint32_t* d_out; CK(cudaMalloc(&d_out, 1 << 20));
-  // baseline shape of round 1: R 24, 2 chains, 256 threads, 2 CTAs/SM
   run<24, 2, 0, 0>("cell", sms, 256, 2, d_out);
   run<24, 2, 1, 0>("cell", sms, 256, 2, d_out);
   run<24, 2, 1, 1>("cell", sms, 256, 2, d_out);
-  run<24, 4, 0, 0>("cell", sms, 256, 2, d_out);
-  run<24, 2, 0, 0>("cell", sms, 256, 1, d_out);
-  run<24, 4, 0, 0>("cell", sms, 256, 1, d_out);
-  // taller lanes, more chains, 1 CTA/SM (up to 255 registers)
-  run<32, 4, 0, 0>("cell", sms, 256, 1, d_out);
-  run<32, 4, 1, 1>("cell", sms, 256, 1, d_out);
+  run<24, 2, 1, 1>("cell", sms, 256, 1, d_out);
+  run<24, 3, 0, 0>("cell", sms, 256, 2, d_out);
+  run<16, 2, 0, 0>("cell", sms, 256, 3, d_out);
+  run<16, 2, 1, 1>("cell", sms, 256, 3, d_out);
+  run<16, 2, 1, 1>("cell", sms, 256, 2, d_out);
+  run<32, 2, 0, 0>("cell", sms, 256, 2, d_out);
+  run<32, 2, 1, 1>("cell", sms, 256, 2, d_out);
   run<32, 4, 1, 1>("cell", sms, 256, 2, d_out);
-  run<48, 4, 0, 0>("cell", sms, 256, 1, d_out);
-  run<48, 4, 1, 0>("cell", sms, 256, 1, d_out);
+  run<24, 2, 1, 1>("cell", sms, 512, 1, d_out);
+  run<24, 2, 1, 1>("cell", sms, 128, 4, d_out);
   run<48, 4, 1, 1>("cell", sms, 256, 1, d_out);
-  run<48, 6, 1, 1>("cell", sms, 256, 1, d_out);
-  run<48, 3, 1, 1>("cell", sms, 256, 1, d_out);
-  run<48, 4, 1, 1>("cell", sms, 384, 1, d_out);
-  run<48, 4, 1, 1>("cell", sms, 128, 2, d_out);
-  run<64, 4, 1, 1>("cell", sms, 256, 1, d_out);
-  run<64, 8, 1, 1>("cell", sms, 256, 1, d_out);
-  run<40, 5, 1, 1>("cell", sms, 256, 1, d_out);
-  run<36, 3, 1, 1>("cell", sms, 384, 1, d_out);
-  run<32, 4, 1, 1>("cell", sms, 384, 1, d_out);
-  run<32, 2, 1, 1>("cell", sms, 384, 1, d_out);
+  run<48, 2, 1, 1>("cell", sms, 256, 1, d_out);
+  run<40, 2, 1, 1>("cell", sms, 256, 1, d_out);
+  run<32, 2, 1, 0>("cell", sms, 256, 2, d_out);
+  run<24, 2, 1, 0>("cell", sms, 384, 1, d_out);
   CK(cudaGetLastError());
   return 0;
 }

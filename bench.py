@@ -43,6 +43,7 @@ WORKLOADS = {
     "c2": "BASELINE config 2: 1 query (567 aa) vs Swiss-Prot-sized synthetic DB (570k seqs, ~205M residues), BLOSUM62, gap 10/2",
     "c1": "BASELINE config 1: 1 query (144 aa) vs 1,000 synthetic sequences, BLOSUM62, gap 10/2",
     "c4": "BASELINE config 4: queries 2,000-35,000 aa vs 1,500 long synthetic sequences (>3,000 aa)",
+    "c5": "BASELINE config 5: 20-query sweep vs TrEMBL-scale synthetic DB (50M seqs, ~16.8G residues)",
     "t5hom": "PAPER Table V homogeneous set: 40 queries 4,500-5,000 aa vs Swiss-Prot-sized synthetic DB (570k seqs)",
     "t5het": "PAPER Table V heterogeneous set: 40 queries 4-35,213 aa vs Swiss-Prot-sized synthetic DB (570k seqs)",
 }
@@ -151,7 +152,7 @@ def config_obj(args, c, q_lens, d_lens, n, n_shards=1):
             **({"gather": "NCCL all-gather of the score blocks, then sw_assemble on rank 0 (caller-order "
                           "scores[Q][N]) inside the timed step"} if n > 1 else {}),
             "l2": "inputs larger than L2: 205 MB packed DB > 126 MB L2, streamed once per query per step"
-            if args.workload in ("c2", "c3", "t5hom", "t5het") and args.n_db is None else "small workload"}
+            if args.workload in ("c2", "c3", "c5", "t5hom", "t5het") and args.n_db is None else "small workload"}
 
 
 def cpu_model() -> str:

@@ -246,6 +246,9 @@ int32_t sw_last_stats(sw_handle_t h, sw_stats_t* out);
  *   "bank_skew"           1: single-query profile copies one per lane group of
  *                         a shared-memory phase at searched bank skews
  *                         (conflict-free; default 1), 0: the linear layout
+ *   "const_gaps"          1 (default): searches with Gs = 10, Ge = 2 use kernel
+ *                         instantiations with the penalties as immediates; 0: the
+ *                         runtime-penalty kernels (same results)
  *   "timing"              1/0, same as SW_FLAG_TIMING
  *   "timing_accumulate"   1: short_ms/long_ms of sw_last_stats sum every search
  *                         since the last "timing_reset" (0: the last search only)

@@ -118,6 +118,9 @@ struct sw_handle_s {
   int64_t opt_pack_queries = 1; // mode-1 slots: fill the shorter half with further queries (strip-aligned)
   int64_t opt_bank_copy = 1;    // query-pair profile: second smem copy shifted by 64 B for odd lane groups
   int64_t opt_bank_skew = 1;    // mode-0 profile copies: per-copy bank skew (mode0_copies)
+  int64_t opt_const_gaps = 1;   // gaps 10/2: the constant-gap kernel instantiations
+  int64_t opt_crit_min = CRIT_MIN_STEPS;                    // long-pair rule (see launch_all)
+  int64_t opt_crit_pct = int64_t(CRIT_FRACTION * 100 + 0.5);
   int64_t opt_align_ws_mb = 2048;  // sw_align: traceback-code workspace per batch
   // sw_align scratch (separate from sw_search's: a search may still be running on another stream)
   DevBuf a_qcodes, a_qoff, a_matrix, a_items, a_links, a_trace, a_best, a_ops, a_out, a_counter;
@@ -355,6 +358,14 @@ int32_t sw_set_option(sw_handle_t h, const char* key, int64_t value) {
     h->opt_bank_copy = value;
   } else if (k == "bank_skew") {
     h->opt_bank_skew = value;
+  } else if (k == "crit_min_steps") {
+    if (value < 1) return set_err(h, SW_EINVAL, "crit_min_steps must be >= 1");
+    h->opt_crit_min = value;
+  } else if (k == "crit_pct") {
+    if (value < 1) return set_err(h, SW_EINVAL, "crit_pct must be >= 1");
+    h->opt_crit_pct = value;
+  } else if (k == "const_gaps") {
+    h->opt_const_gaps = value;
   } else if (k == "query_pairs") {
     h->opt_query_pairs = value;
   } else if (k == "timing_accumulate") {
@@ -622,7 +633,7 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
     group_steps += double(sl.strips) * (cols + seqs * VG);
   }
   resident_groups = 2.0 * h->sms * double(!m1.empty() ? NG1 : NG0);
-  const double crit = std::max(double(CRIT_MIN_STEPS), CRIT_FRACTION * group_steps / resident_groups);
+  const double crit = std::max(double(h->opt_crit_min), 0.01 * double(h->opt_crit_pct) * group_steps / resident_groups);
   // Long-sequence databases (most residues in pairs longer than T_LONG, config 4)
   // are scored entirely by the intra-task kernel; otherwise the critical-path
   // rule alone decides.
@@ -908,7 +919,8 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
     }
     const bool with_long = combined && mode == 0;
     if (with_long) smem = std::max(smem, smem_long);  // an item is short or long: the two uses share smem
-    const int occ = with_long ? combined_max_ctas_per_sm(G, R, smem) : short_max_ctas_per_sm(mode, G, R, smem);
+    const bool cg = c.nGe == 0xfffefffeu && c.nGsGe == 0xfff4fff4u && h->opt_const_gaps != 0;
+    const int occ = with_long ? combined_max_ctas_per_sm(G, R, smem) : short_max_ctas_per_sm(mode, G, R, smem, cg);
     if (occ <= 0) fail(SW_ECUDA, "short-pair kernel does not fit on an SM");
     const int64_t items = int64_t(n_short) + (with_long ? long_items : 0);
     const int grid = int(std::max<int64_t>(1, std::min<int64_t>(items, int64_t(occ) * h->sms)));
@@ -938,7 +950,7 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
       al.wrap = h->wrap.as<uint2>();
       SW_CK(launch_combined(G, R, grid, smem, as, al, c.st));
     } else {
-      SW_CK(launch_short(mode, G, R, grid, smem, as, c.st));
+      SW_CK(launch_short(mode, G, R, grid, smem, as, c.st, cg));
     }
     if (ev) SW_CK(cudaEventRecord(ev->second, c.st));
     ++out.launches;

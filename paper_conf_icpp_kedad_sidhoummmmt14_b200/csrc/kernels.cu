@@ -361,8 +361,12 @@ __device__ __forceinline__ void stage_issue(ProfStage& ps, int b, int tag, const
   ps.pending |= 1u << b;
 }
 
-template <int G, int R, int NT, bool Q2>
+// CG: the gap penalties are the compile-time pair Gs = 10, Ge = 2 (BASELINE's
+// configuration): the cell update then encodes -Ge and -(Gs+Ge) as immediates,
+// one register operand fewer per VIADDMNMX / VIADD (register-file bandwidth).
+template <int G, int R, int NT, bool Q2, bool CG = false>
 __device__ __forceinline__ void short_item(const ShortArgs& a, int item, uint8_t* smem, int& loaded, ProfStage& ps) {
+  const uint32_t nGe = CG ? 0xfffefffeu : a.nGe, nGsGe = CG ? 0xfff4fff4u : a.nGsGe;
   uint8_t* sprof = smem;                         // the strip profile (bank-spread copies)
   constexpr int NG = NT / G;
   const int tid = threadIdx.x;
@@ -427,7 +431,7 @@ __device__ __forceinline__ void short_item(const ShortArgs& a, int item, uint8_t
           __syncwarp();
         }
         strip_pass<G, R, false, true>(gprof, a.LS, a.LB, a.stream + pr.off, pr.len, T, k, rd, s + 1 < d.n_strips,
-                                      bb, bb, Chain{}, a.code_pad2, a.nGe, a.nGsGe, best, half ? 8u : 0u);
+                                      bb, bb, Chain{}, a.code_pad2, nGe, nGsGe, best, half ? 8u : 0u);
         if (si.emit0 >= 0 || si.emit1 >= 0) {  // a query of either half ends with this strip
           uint32_t bg = best;
 #pragma unroll
@@ -449,7 +453,7 @@ __device__ __forceinline__ void short_item(const ShortArgs& a, int item, uint8_t
         }
       } else {
         strip_pass<G, R, false>(gprof, a.LS, a.LB, a.stream + pr.off, pr.len, T, k, s > 0, s + 1 < d.n_strips,
-                                bb, bb, Chain{}, a.code_pad2, a.nGe, a.nGsGe, best);
+                                bb, bb, Chain{}, a.code_pad2, nGe, nGsGe, best);
       }
     }
     if constexpr (!Q2) {  // mode 0: one query, both halves are DB sequences
@@ -585,7 +589,7 @@ __device__ __forceinline__ void long_item(const LongArgs& a, int item, uint8_t* 
 // The short-pair kernel: one persistent launch per short-pair mode (query pairs,
 // single query), one (G, R) per launch, its own register budget (the query-pair
 // form keeps R = 32 rows per lane at 128 registers, 2 CTAs per SM).
-template <int G, int R, int NT, bool Q2>
+template <int G, int R, int NT, bool Q2, bool CG = false>
 __global__ void __launch_bounds__(NT, 2) short_kernel(ShortArgs as) {
   extern __shared__ __align__(128) uint8_t smem[];
   __shared__ int s_item;
@@ -603,7 +607,7 @@ __global__ void __launch_bounds__(NT, 2) short_kernel(ShortArgs as) {
     const int item = s_item;
     __syncthreads();
     if (item >= as.n_items) break;
-    short_item<G, R, NT, Q2>(as, item, smem, loaded, ps);
+    short_item<G, R, NT, Q2, CG>(as, item, smem, loaded, ps);
   }
 }
 
@@ -667,7 +671,21 @@ typedef void (*short_fn)(ShortArgs);
   X(16, 8) X(16, 12) X(16, 16) X(16, 20) X(16, 24) X(16, 28) X(16, 32)             \
   X(32, 8) X(32, 12) X(32, 16) X(32, 20) X(32, 24) X(32, 28) X(32, 32)
 
-static short_fn pick_short(int mode, int G, int R) {
+// constant-gap (Gs 10, Ge 2) instantiations of the geometries the cost model picks
+// for Swiss-Prot-like databases
+#define SW_CG_CASES(X) X(4, 32) X(4, 24) X(8, 32) X(8, 24) X(4, 16) X(8, 16)
+
+static short_fn pick_short(int mode, int G, int R, bool cg = false) {
+  if (cg && mode == 1) {
+#define X(g, r) if (G == g && R == r) return short_kernel<g, r, SCORE_NT, true, true>;
+    SW_CG_CASES(X)
+#undef X
+  }
+  if (cg && mode == 0) {
+#define X(g, r) if (G == g && R == r) return short_kernel<g, r, SCORE_NT, false, true>;
+    SW_CG_CASES(X)
+#undef X
+  }
   if (mode == 1) {
 #define X(g, r) if (G == g && R == r) return short_kernel<g, r, SCORE_NT, true>;
     SW_GEOM_CASES(X)
@@ -689,13 +707,16 @@ static int occupancy(const void* f, int threads, int smem_bytes) {
   return n;
 }
 
-int short_max_ctas_per_sm(int mode, int G, int R, int smem_bytes) {
-  short_fn f = pick_short(mode, G, R);
+int short_max_ctas_per_sm(int mode, int G, int R, int smem_bytes, bool cg) {
+  short_fn f = pick_short(mode, G, R, cg);
+  if (!f) f = pick_short(mode, G, R);
   return f ? occupancy(reinterpret_cast<const void*>(f), SCORE_NT, smem_bytes) : 0;
 }
 
-cudaError_t launch_short(int mode, int G, int R, int grid, int smem_bytes, const ShortArgs& a, cudaStream_t st) {
-  short_fn f = pick_short(mode, G, R);
+cudaError_t launch_short(int mode, int G, int R, int grid, int smem_bytes, const ShortArgs& a, cudaStream_t st,
+                         bool cg) {
+  short_fn f = pick_short(mode, G, R, cg);
+  if (!f) f = pick_short(mode, G, R);
   if (!f) return cudaErrorInvalidValue;
   if (smem_bytes > 48 * 1024) {
     cudaError_t e = cudaFuncSetAttribute(f, cudaFuncAttributeMaxDynamicSharedMemorySize, smem_bytes);

@@ -186,8 +186,10 @@ cudaError_t launch_build_profile_q2(const uint8_t* qa, int ma, const uint8_t* qb
 constexpr int SCORE_NT = 256;       // threads per CTA of both
 constexpr int LONG_W = SCORE_NT / 32;
 bool short_config_supported(int mode, int G, int R);
-int short_max_ctas_per_sm(int mode, int G, int R, int smem_bytes);
-cudaError_t launch_short(int mode, int G, int R, int grid, int smem_bytes, const ShortArgs& a, cudaStream_t st);
+// cg: the gaps are Gs = 10, Ge = 2 -- use the constant-gap instantiation when one exists
+int short_max_ctas_per_sm(int mode, int G, int R, int smem_bytes, bool cg = false);
+cudaError_t launch_short(int mode, int G, int R, int grid, int smem_bytes, const ShortArgs& a, cudaStream_t st,
+                         bool cg = false);
 int long_max_ctas_per_sm(int smem_bytes);
 // single-query searches with long pairs: long items and mode-0 short items in one launch
 int combined_max_ctas_per_sm(int G, int R, int smem_bytes);

@@ -464,3 +464,16 @@ def test_overflow_threshold_is_clamped():
     ref = oracle_scores(q, np.array([0, len(q)], np.int64), dc, do)
     assert ref.max() > 32767
     np.testing.assert_array_equal(got, ref)
+
+
+@pytest.mark.parametrize("cg", [0, 1])
+@pytest.mark.parametrize("pairs", [0, 1])
+def test_constant_gap_kernels(cg, pairs):
+    """Gs = 10, Ge = 2 searches run the constant-gap instantiations (penalties as
+    immediates) unless option const_gaps is 0; both give the oracle's scores,
+    multi-strip queries included."""
+    rng = np.random.default_rng(95 + 2 * cg + pairs)
+    dc, do = _seqs(list(rng.integers(1, 500, size=150)) + [0, 1, 3], rng)
+    qc, qo = _seqs([700, 129, 64, 3100, 2], rng)
+    got = gpu_scores(qc, qo, dc, do, opts={"const_gaps": cg, "query_pairs": pairs})
+    np.testing.assert_array_equal(got, oracle_scores(qc, qo, dc, do))

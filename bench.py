@@ -8,8 +8,8 @@ intra-task DPX kernels, int32 re-score) plus, at N > 1, the single collective
 into scores[Q][N] in the caller's order -- dist.ShardedSearch.step().  Workload (default): BASELINE config 3, the 20-query
 sweep (144..5478 aa) against the Swiss-Prot-sized synthetic DB (570k seqs,
 205M residues) -- the configuration the metric "GCUPS at 1/2/4/8 B200" is
-quoted on; at N > 1 the DB is cut into 4N shards whose (query, shard) tasks are
-placed on the GPUs by the dual approximation.
+quoted on; at N > 1 the DB is cut into N equal-residue shards, placed on the
+GPUs by the dual approximation as whole-shard tasks (one search per GPU).
 
   python bench.py [--gpus N] [--steps K] [--warmup W] [--impl ours|reference]
   torchrun --nproc-per-node N bench.py --gpus N ...
@@ -72,7 +72,9 @@ def parse():
     ap.add_argument("--force-geom", default=None, help="G,R of the inter-task kernel (experiments; default auto)")
     ap.add_argument("--verify", type=int, default=0, help="after timing, check N sampled DB sequences "
                     "of the assembled scores against the CPU oracle (rank 0)")
-    ap.add_argument("--shards", type=int, default=None, help="DB shards (default: 1 at N = 1, 4 per GPU at N > 1)")
+    ap.add_argument("--shards", type=int, default=None, help="DB shards (default: one per GPU)")
+    ap.add_argument("--tasks", default="shard", choices=["shard", "pair"],
+                    help="placement tasks: whole shards (default) or (query, shard) pairs")
     ap.add_argument("--dist-backend", default="nccl", help="nccl (default); gloo only for functional checks "
                     "of the multi-rank path on a box with fewer GPUs than ranks")
     return ap.parse_args()
@@ -148,7 +150,7 @@ def config_obj(args, c, q_lens, d_lens, n, n_shards=1):
             "n_queries": int(len(q_lens)), "query_residues": int(q_lens.sum()),
             "n_db_seqs": int(len(d_lens)), "db_residues": int(d_lens.sum()),
             "matrix": "BLOSUM62", "gap_open": 10, "gap_extend": 2,
-            "shards": n_shards, "placement": "dual-approximation (query, shard) tasks, calibrated task times",
+            "shards": n_shards, "placement": f"dual approximation over {args.tasks} tasks, calibrated task times",
             **({"gather": "NCCL all-gather of the score blocks, then sw_assemble on rank 0 (caller-order "
                           "scores[Q][N]) inside the timed step"} if n > 1 else {}),
             "l2": "inputs larger than L2: 205 MB packed DB > 126 MB L2, streamed once per query per step"
@@ -292,7 +294,7 @@ def run_ours(args):
         h.set_option("force_R", fr)
     # the multi-GPU path (and, at N = 1, the single search): dist.ShardedSearch
     ss = swdist.ShardedSearch(h, c["dcodes"], c["doff"], c["qcodes"], c["qoff"], S, 10, 2, rank=rank, world=world,
-                              n_shards=args.shards, pg=pg, backend=args.dist_backend)
+                              n_shards=args.shards, pg=pg, backend=args.dist_backend, tasks=args.tasks)
     stream = torch.cuda.current_stream(dev)
 
     for _ in range(args.warmup):

@@ -113,6 +113,32 @@ def _place(q_lens, shards, n_gpus, rate, tasks, res) -> Plan:
     return plan
 
 
+def place_shards(q_lens, shards, shard_residues, n_gpus: int) -> Plan:
+    """Dual-approximation placement of SHARD tasks: task s = every query against
+    shard s (the paper's task is a query against the whole database, L304-305;
+    with the database cut into shards the coarsest task is a shard with the whole
+    query set).  One sw_search per task: with S = k equal-residue shards each GPU
+    runs ONE search over 1/k of the database, the most efficient launch shape
+    (measured: (query, shard) tasks on 4k shards scatter into ~30 small searches
+    per GPU at k = 8 and run at a third of the single-search rate,
+    profiles/r02_shard_probe.jsonl)."""
+    q_lens = [int(x) for x in q_lens]
+    res = [float(r) for r in shard_residues]
+    p_gpu = np.array([sum(gpu_task_time(m, res[s]) for m in q_lens) for s in range(len(shards))], dtype=np.float64)
+    if len(shards):
+        pe, mk, lam = schedule_dual(p_gpu * 1e6, p_gpu, 0, n_gpus)
+    else:
+        pe, mk, lam = np.zeros(0, np.int32), 0.0, 0.0
+    tasks = [(q, s) for s in range(len(shards)) for q in range(len(q_lens))]
+    owner = np.array([int(pe[s]) for s in range(len(shards)) for _q in range(len(q_lens))], dtype=np.int64)
+    plan = Plan(n_gpus=n_gpus, shards=shards, tasks=tasks, owner=owner, makespan=mk, lam=lam)
+    for g in range(n_gpus):
+        plan.by_gpu[g] = {}
+    for (q, s), g in zip(tasks, plan.owner):
+        plan.by_gpu[int(g)].setdefault(s, []).append(q)
+    return plan
+
+
 def local_blocks(plan: Plan, rank: int):
     """Ordered list of (shard, queries) this rank scores; defines the flat layout."""
     d = plan.by_gpu.get(rank, {})
@@ -168,10 +194,12 @@ class ShardedSearch:
     tests run THIS code path.
 
     Setup (untimed, like a resident search service): the DB is cut into
-    n_shards snake-dealt shards (default 4 per GPU), the (query, shard) tasks are
-    placed by the dual approximation (sw_schedule_dual, calibrated task times),
-    this rank loads the shards its tasks reference and prepares one sw_search
-    per (shard, query list) block into a flat device buffer.
+    n_shards snake-dealt shards of equal residues (default one per GPU); the
+    tasks -- whole shards with every query (tasks="shard", default) or (query,
+    shard) pairs (tasks="pair") -- are placed by the dual approximation
+    (sw_schedule_dual, calibrated task times); this rank loads the shards its
+    tasks reference and prepares one sw_search per (shard, query list) block
+    into a flat device buffer.
     step(): the rank's searches, then -- the single data-path exchange -- the
     all-gather of the flat blocks (NCCL over NVLink; gloo with host staging for
     functional runs), then on rank 0 sw_assemble merges them into scores[Q][N]
@@ -180,18 +208,21 @@ class ShardedSearch:
     """
 
     def __init__(self, handle, dcodes, doff, qcodes, qoff, matrix, gap_open=10, gap_extend=2, rank=0, world=1,
-                 n_shards=None, pg=None, backend="nccl", alphabet_size=24, rate=None):
+                 n_shards=None, pg=None, backend="nccl", alphabet_size=24, rate=None, tasks="shard"):
         import torch
         self.h, self.rank, self.world, self.pg, self.backend = handle, rank, world, pg, backend
         self.matrix, self.gs, self.ge = matrix, gap_open, gap_extend
         doff = np.asarray(doff, dtype=np.int64)
         qoff = np.asarray(qoff, dtype=np.int64)
         self.Q, self.N = len(qoff) - 1, len(doff) - 1
-        n_shards = n_shards or (4 * world if world > 1 else 1)
+        n_shards = n_shards or world
         self.shards = shard_cut(doff, n_shards)
         lens = np.diff(doff)
         res = [int(lens[s].sum()) for s in self.shards]
-        self.plan = place(np.diff(qoff), self.shards, res, world, rate=rate)
+        if tasks == "shard":
+            self.plan = place_shards(np.diff(qoff), self.shards, res, world)
+        else:  # (query, shard) tasks
+            self.plan = place(np.diff(qoff), self.shards, res, world, rate=rate)
         self.blocks = local_blocks(self.plan, rank)
         dev = torch.device("cuda", handle.device)
         self.dev = dev

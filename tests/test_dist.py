@@ -194,9 +194,28 @@ def test_assembly_tables_match_assemble(world, shards):
 
 def test_task_time_model_orders_by_padded_rows():
     """Calibrated GPU task times: strip-padded rows x residues
-    / rate + a fixed share; a 144-row query costs as much as a 192-row one."""
+    / rate + a fixed share; a query costs as much as its strip-padded height."""
     t = swdist.gpu_task_time
-    assert t(144, 1e6) == t(192, 1e6)
-    assert t(193, 1e6) > t(192, 1e6)
+    S = swdist.STRIP_ROWS
+    assert t(S + 16, 1e6) == t(2 * S, 1e6)
+    assert t(2 * S + 1, 1e6) > t(2 * S, 1e6)
     assert t(0, 1e6) == 0.0 and t(100, 0) == 0.0
     assert abs(t(9600, 1e8) - (9600 * 1e8 / swdist.RATE + swdist.T_TASK)) < 1e-12
+
+
+@pytest.mark.parametrize("k", [1, 2, 3, 8])
+def test_place_shards_one_search_per_gpu(k):
+    """Shard tasks (every query against one shard): with S = k equal-residue
+    shards the dual approximation gives each GPU exactly one shard (one search);
+    every (query, shard) pair is covered once; the makespan is the largest
+    shard's modelled time."""
+    c = swgen.make_config("c3", n_db=4000)
+    ql = np.diff(c["qoff"])
+    sh = swdist.shard_cut(c["doff"], k)
+    res = [int(np.diff(c["doff"])[s].sum()) for s in sh]
+    plan = swdist.place_shards(ql, sh, res, k)
+    seen = sorted((q, s) for r in range(k) for s, qs in swdist.local_blocks(plan, r) for q in qs)
+    assert seen == sorted((q, s) for q in range(len(ql)) for s in range(k))
+    assert all(len(swdist.local_blocks(plan, r)) == 1 for r in range(k))
+    per = [sum(swdist.gpu_task_time(m, res[s]) for m in ql) for s in range(k)]
+    assert plan.makespan == pytest.approx(max(per))

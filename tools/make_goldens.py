@@ -86,6 +86,31 @@ def full_config(name, procs):
         "rows": [row_record(i, ref[i]) for i in range(nq)]})
 
 
+_G = {}
+
+
+def _rows_worker(args):
+    """One slice of the DB against one query, in a forked worker: the DB arrays are
+    inherited from the parent (module global), never pickled (C5's are 17 GB)."""
+    qi, b0, b1 = args
+    c = _G["c"]
+    qc = np.ascontiguousarray(c["qcodes"][c["qoff"][qi]:c["qoff"][qi + 1]])
+    qo = np.array([0, len(qc)], dtype=np.int64)
+    off = c["doff"][b0:b1 + 1]
+    dc = c["dcodes"][int(off[0]):int(off[-1])]
+    return qi, b0, oracle.gotoh_search(qc, qo, dc, off - off[0], _G["S"], 10, 2, procs=1)[0]
+
+
+def _pairs_worker(args):
+    """Oracle scores of sampled (query, sequence) pairs of one query (forked worker)."""
+    qi, ids = args
+    c = _G["c"]
+    sc, so = swgen.subset(c["dcodes"], c["doff"], ids)
+    qc = np.ascontiguousarray(c["qcodes"][c["qoff"][qi]:c["qoff"][qi + 1]])
+    qo = np.array([0, len(qc)], dtype=np.int64)
+    return qi, ids, oracle.gotoh_search(qc, qo, sc, so, _G["S"], 10, 2, procs=1)[0]
+
+
 def c5(procs, n_db=None):
     t0 = time.time()
     c = swgen.make_config("c5", n_db=n_db)
@@ -94,26 +119,41 @@ def c5(procs, n_db=None):
     print(f"c5: {nq} queries x {nd} seqs, {int(c['doff'][-1])} residues, generated in "
           f"{time.time() - t0:.1f}s", flush=True)
     S = blosum62()
-    # (i) the m = 144 query (query 0) against the whole DB
+    import multiprocessing as mp
+    _G["c"], _G["S"] = c, S
+    oracle.build()
+    ctx = mp.get_context("fork")
+    # (i) the m = 144 query (query 0) against the whole DB, in residue-balanced slices
     t1 = time.time()
-    q0c = np.ascontiguousarray(c["qcodes"][c["qoff"][0]:c["qoff"][1]])
-    q0o = np.array([0, len(q0c)], dtype=np.int64)
-    row = oracle.gotoh_search(q0c, q0o, c["dcodes"], c["doff"], S, 10, 2, procs=procs)[0]
+    cum = c["doff"][1:] - c["doff"][0]
+    nchunks = procs * 16
+    cuts = sorted(set([0] + [int(np.searchsorted(cum, int(cum[-1]) * k // nchunks)) for k in range(1, nchunks)]
+                      + [nd]))
+    row = np.zeros(nd, dtype=np.int32)
+    with ctx.Pool(procs) as pool:
+        for _qi, b0, part in pool.imap_unordered(_rows_worker, [(0, a, b) for a, b in zip(cuts[:-1], cuts[1:]) if b > a]):
+            row[b0:b0 + len(part)] = part
     t_row = time.time() - t1
     print(f"c5 query-0 row in {t_row:.0f}s", flush=True)
     # (ii) stratified sample, (iii) planted pairs
     smp = swgen.c5_sample(c["doff"], nq)
     t1 = time.time()
     scores = np.zeros(len(smp["q"]), dtype=np.int32)
+    jobs = []
     for qi in range(nq):
         sel = np.nonzero(smp["q"] == qi)[0]
-        if not len(sel):
-            continue
-        ids = smp["d"][sel]
-        sc, so = swgen.subset(c["dcodes"], c["doff"], ids)
-        qc = np.ascontiguousarray(c["qcodes"][c["qoff"][qi]:c["qoff"][qi + 1]])
-        qo = np.array([0, len(qc)], dtype=np.int64)
-        scores[sel] = oracle.gotoh_search(qc, qo, sc, so, S, 10, 2, procs=procs)[0]
+        for part in np.array_split(sel, procs):
+            if len(part):
+                jobs.append((qi, smp["d"][part]))
+    pos = {}
+    for qi in range(nq):
+        sel = np.nonzero(smp["q"] == qi)[0]
+        for k, d in enumerate(smp["d"][sel]):
+            pos[(qi, int(d))] = int(sel[k])
+    with ctx.Pool(procs) as pool:
+        for qi, ids, vals in pool.imap_unordered(_pairs_worker, jobs):
+            for d, v in zip(ids, vals):
+                scores[pos[(qi, int(d))]] = v
     t_smp = time.time() - t1
     smp["cells"] = float((np.diff(c["qoff"])[smp["q"]] * np.diff(c["doff"])[smp["d"]]).sum())
     strata = {}

@@ -9,12 +9,13 @@ import swgen  # noqa: E402
 import paper_conf_icpp_kedad_sidhoummmmt14_b200 as sw  # noqa: E402
 from paper_conf_icpp_kedad_sidhoummmmt14_b200 import dist  # noqa: E402
 
-k = int(sys.argv[1]); S = int(sys.argv[2]) if len(sys.argv) > 2 else 4 * k
+k = int(sys.argv[1]); S = int(sys.argv[2]) if len(sys.argv) > 2 else k
+mode = sys.argv[3] if len(sys.argv) > 3 else "shard"
 c = swgen.make_config("c3")
 ql = np.diff(c["qoff"])
 sh = dist.shard_cut(c["doff"], S)
 res = [int(np.diff(c["doff"])[s].sum()) for s in sh]
-plan = dist.place(ql, sh, res, k)
+plan = dist.place_shards(ql, sh, res, k) if mode == "shard" else dist.place(ql, sh, res, k)
 with sw.Handle(0, timing=True) as h:
     for kv in filter(None, os.environ.get("SWDUAL_OPTS", "").split(",")):
         h.set_option(kv.split("=")[0], int(kv.split("=")[1]))
@@ -32,7 +33,7 @@ with sw.Handle(0, timing=True) as h:
             e1.record()
             torch.cuda.synchronize()
             times.append(e0.elapsed_time(e1) / 1e3)
-print(json.dumps({"k": k, "shards": S, "opts": os.environ.get("SWDUAL_OPTS", ""), "model_s": plan.makespan,
+print(json.dumps({"k": k, "shards": S, "tasks": mode, "opts": os.environ.get("SWDUAL_OPTS", ""), "model_s": plan.makespan,
                   "measured_max_s": max(times), "measured_sum_s": sum(times),
                   "eff_GCUPS_sum": float(ql.sum()) * float(c["doff"][-1]) / sum(times) / 1e9,
                   "searches": sum(len(jobs[r]) for r in range(k))}), flush=True)

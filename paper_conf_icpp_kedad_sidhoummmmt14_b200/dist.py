@@ -68,15 +68,16 @@ class Plan:
 
 # GPU time model of one (query, shard) task on a B200 (p_j from a
 # calibrated rate).  The scoring kernel sweeps whole strips of STRIP_ROWS query
-# rows (the geometry chosen for Swiss-Prot-like DBs), so a query of m residues
-# costs ceil(m / STRIP_ROWS) * STRIP_ROWS rows -- which is why short queries run
-# at a lower cell rate (the per-query rates measured in
-# profiles/r01_hybrid_probe.jsonl: 144 aa ~0.75 of the long-query rate); plus a
-# per-task share of the launch and its tail.  RATE: the long-query cell rate of
-# the C3 bench (profiles/r01_end_bench_c3.json).
-STRIP_ROWS = 96
-RATE = 6.9e12          # computed cells per second per B200
-T_TASK = 5.0e-5        # seconds per task (profile build, launch tail share)
+# rows (the query-pair geometry chosen for Swiss-Prot-like databases, G = 4 lanes
+# x R = 32 rows), so a query of m residues costs ceil(m / STRIP_ROWS) * STRIP_ROWS
+# rows -- which is why short queries run at a lower cell rate -- plus a per-task
+# share of the search's fixed cost (launch tail, long-pair critical path).
+# Calibrated on C3 in the k = 2 and k = 8 whole-shard layouts
+# (profiles/r02_shard_probe.jsonl): t(k) = A / k + c with A = 1.115 s, c = 9.6 ms
+# per 20-query search.
+STRIP_ROWS = 128
+RATE = 7.9e12          # strip-padded cells per second per B200
+T_TASK = 4.8e-4        # seconds per task
 
 
 def gpu_task_time(m: int, residues: float) -> float:

@@ -98,6 +98,7 @@ struct sw_handle_s {
   DevBuf qcodes, qoff, matrix, prof, bbuf1, bbuf0, wrap, counters, ovf, ovf_count, scores_tmp, rbuf, qdesc;
   DevBuf rgrows, rflags;  // re-score: CTA-to-CTA rows, counters
   DevBuf imap;            // short work item order (mode 1 items, then mode 0 items)
+  DevBuf lmap;            // long work item order
   DevBuf vq, sinfo;       // packed mode-1 slots: strip-padded query codes per half, per-strip info
   cudaStream_t side = nullptr;             // the long-pair kernel's stream when short pairs run too
   cudaEvent_t ev_fork = nullptr, ev_join = nullptr;
@@ -693,6 +694,8 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
   const bool combined = any_long && any_m0 && !any_q2;
   // ---- long work: one item per (query, long pair), or per `pack` pairs
   std::vector<LongQuery> ldesc;
+  struct LItem { double cost; int q, it; };
+  std::vector<LItem> litems;
   int64_t long_items = 0;
   int32_t max_long = 0;
   for (size_t k = 0; k < order.size(); ++k) {
@@ -705,9 +708,13 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
     d.scores = c.dscores + int64_t(order[k]) * db->out_n;
     d.n_strips = gl[k].n_strips;
     d.qidx = order[k];
-    d.item_begin = int(long_items);
     d.n_long = nl;
     d.pack = (combined || gl[k].n_strips >= W) ? 1 : W / gl[k].n_strips;
+    // item cost: rounds x the item's longest pair (pairs are sorted longest first)
+    const int GS = gl[k].n_strips >= W ? W : gl[k].n_strips;
+    const double rounds = double((gl[k].n_strips + GS - 1) / GS);
+    for (int it = 0; it * d.pack < nl; ++it)
+      litems.push_back({rounds * double(db->pairs[size_t(it * d.pack)].len + 64), int(ldesc.size()), it});
     ldesc.push_back(d);
     long_items += (nl + d.pack - 1) / d.pack;
     max_long = std::max(max_long, db->pairs[0].len);
@@ -823,6 +830,13 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
   SW_CK(h->imap.ensure(std::max<size_t>(imap.size(), 1) * sizeof(int2)));
   if (!imap.empty())
     SW_CK(cudaMemcpyAsync(h->imap.p, imap.data(), imap.size() * sizeof(int2), cudaMemcpyHostToDevice, c.st));
+  // long items costliest first across all queries (so no big item starts late)
+  std::stable_sort(litems.begin(), litems.end(), [](const LItem& x, const LItem& y) { return x.cost > y.cost; });
+  std::vector<int2> lmap(litems.size());
+  for (size_t i = 0; i < litems.size(); ++i) lmap[i] = make_int2(litems[i].q, litems[i].it);
+  SW_CK(h->lmap.ensure(std::max<size_t>(lmap.size(), 1) * sizeof(int2)));
+  if (!lmap.empty())
+    SW_CK(cudaMemcpyAsync(h->lmap.p, lmap.data(), lmap.size() * sizeof(int2), cudaMemcpyHostToDevice, c.st));
   SW_CK(h->qdesc.ensure(ldesc.size() * sizeof(LongQuery) + sdesc.size() * sizeof(SlotDesc) + 16));
   LongQuery* d_ldesc = h->qdesc.as<LongQuery>();
   SlotDesc* d_slots = reinterpret_cast<SlotDesc*>(h->qdesc.as<uint8_t>() + ldesc.size() * sizeof(LongQuery));
@@ -849,6 +863,7 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
     al.queries = d_ldesc;
     al.n_queries = int(ldesc.size());
     al.n_items = int(long_items);
+    al.lmap = h->lmap.as<int2>();
     al.SBL = l0.SB; al.LSL = l0.LS; al.LBL = l0.LB;
     smem_long = (W - 1) * LONG_RING * int(sizeof(uint2)) + W * l0.SB;
     al.wcap = max_long + 64 + 8;

@@ -506,19 +506,15 @@ __device__ __forceinline__ void long_item(const LongArgs& a, int item, uint8_t* 
   {
     if (tid < W) { s_prog[tid] = -1; s_cons[tid] = 0; s_best[tid] = 0; }
     __syncthreads();
-    int lo = 0, hi = a.n_queries - 1;
-    while (lo < hi) {
-      const int mid = (lo + hi + 1) >> 1;
-      if (a.queries[mid].item_begin <= item) lo = mid; else hi = mid - 1;
-    }
-    const LongQuery d = a.queries[lo];
+    const int2 li = a.lmap[item];  // (query, item within the query), costliest first across queries
+    const LongQuery d = a.queries[li.x];
     const int ns = d.n_strips;
     // a query of fewer strips than warps: P (host-chosen, <= W / ns) pairs per item, ns warps each
     const int P = d.pack;
     const int GS = ns >= W ? W : ns;             // warps per pair
     const int grp = warp / GS, wg = warp - grp * GS;
     const int j = GS - 1 - wg;                   // position of this warp's strip within a round
-    const int pidx = (item - d.item_begin) * P + grp;
+    const int pidx = li.y * P + grp;
     const bool active = grp < P && pidx < d.n_long;
     PairRec pr;
     if (active) pr = a.pairs[pidx];
@@ -569,7 +565,7 @@ __device__ __forceinline__ void long_item(const LongArgs& a, int item, uint8_t* 
     if (lane == 0) s_best[warp] = best;
     __syncthreads();
     if (tid < P) {
-      const int pj = (item - d.item_begin) * P + tid;
+      const int pj = li.y * P + tid;
       if (pj < d.n_long) {
         const PairRec pq = a.pairs[pj];
         uint32_t b = 0;

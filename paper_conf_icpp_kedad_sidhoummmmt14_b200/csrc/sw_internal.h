@@ -64,17 +64,16 @@ struct LongQuery {
   int32_t* scores;           // this query's row of scores[Q][N] (caller order)
   int n_strips;
   int qidx;
-  int item_begin;            // first long item of this query
   int n_long;
   int pack;                  // pairs per item: 1, or up to W / n_strips when n_strips < W (the
                              // CTA's warps then chain several pairs side by side)
-  int pad_;
 };
 
 struct LongArgs {
   const LongQuery* queries;  // [n_queries], processing order
   int n_queries;
-  int n_items;               // sum of n_long
+  int n_items;               // long items of the launch
+  const int2* lmap;          // item -> (query, item within the query), costliest first
   int SBL, LSL, LBL;         // long profile geometry
   uint2* wrap;               // [gridDim][wcap]: the round-wrap link row of each CTA (warp W-1 -> warp 0)
   int wcap;

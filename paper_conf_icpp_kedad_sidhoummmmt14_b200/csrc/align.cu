@@ -77,7 +77,7 @@ __global__ void __launch_bounds__(ALIGN_WARPS * 32) align_fwd_kernel(AlignArgs a
   int2* __restrict__ links = a.links + ((size_t)blockIdx.x * ALIGN_WARPS + size_t(team) * TW) * a.bcap;
   const int pad = a.alpha;
   const int nGe = -a.Ge, nGsGe = -(a.Gs + a.Ge);
-  const uint32_t padw = uint32_t(pad) * 0x01010101u;
+  const uint2 padw = pad_codes4(pad, a.nib);
   __syncthreads();  // matrix staged
   for (;;) {
     team_sync<TW>();
@@ -106,9 +106,9 @@ __global__ void __launch_bounds__(ALIGN_WARPS * 32) align_fwd_kernel(AlignArgs a
     const int m = int(a.qoff[it.q + 1] - a.qoff[it.q]);
     const int L = (it.n + 3) & ~3;  // this sequence's columns, in whole 4-column words
     const int T = L + 32;           // steps per strip (= trace words per lane per strip)
-    const uint32_t shift = it.half ? 8u : 0u;
+    const int half = it.half;
     const int nstrips = (m + 32 * R - 1) / (32 * R);
-    const uint2* __restrict__ codes = reinterpret_cast<const uint2*>(a.stream + pr.off);
+
     uint32_t* __restrict__ trace = a.trace + it.trace_off;
     const int jw = W - 1 - warp;  // producers on higher warp ids
     Best acc{0, 0x7fffffff, 0x7fffffff};
@@ -152,13 +152,13 @@ __global__ void __launch_bounds__(ALIGN_WARPS * 32) align_fwd_kernel(AlignArgs a
       int hdiag = 0, sH = 0, sF = 0, sC = pad;
       uint32_t eob = 0;  // bit rr: E of this column's row rr was opened (from H of the previous column)
       const int2 z2 = make_int2(0, 0);
-      uint2 cw = make_uint2(padw, padw);
+      uint2 cw = padw;
       int2 tb0 = z2, tb1 = z2, tb2 = z2, tb3 = z2;
       int seen = -1;
       Best sb{0, 0x7fffffff, 0x7fffffff};  // this strip's best of this lane (first hit in (j, i) order)
       if (rd) wait_progress(lk, lk.in_base + min(4 + 31 + ALIGN_LAG, L + 32), seen);
       if (lead) {
-        cw = codes[0];
+        cw = load_codes4(a.stream, pr.off, 0, a.nib);
         if (rd) { tb0 = __ldcg(rp + 0); tb1 = __ldcg(rp + 1); tb2 = __ldcg(rp + 2); tb3 = __ldcg(rp + 3); }
       }
       __syncwarp();
@@ -168,12 +168,12 @@ __global__ void __launch_bounds__(ALIGN_WARPS * 32) align_fwd_kernel(AlignArgs a
         if (rd && t0 + 4 < L) wait_progress(lk, lk.in_base + min(t0 + 8 + 31 + ALIGN_LAG, L + 32), seen);
         if (lead) {
           if (t0 + 4 < L) {
-            cw = codes[(t0 + 4) >> 2];
+            cw = load_codes4(a.stream, pr.off, t0 + 4, a.nib);
             if (rd) {
               tb0 = __ldcg(rp + t0 + 4); tb1 = __ldcg(rp + t0 + 5); tb2 = __ldcg(rp + t0 + 6); tb3 = __ldcg(rp + t0 + 7);
             }
           } else {
-            cw = make_uint2(padw, padw);
+            cw = padw;
             tb0 = z2; tb1 = z2; tb2 = z2; tb3 = z2;
           }
         }
@@ -184,8 +184,7 @@ __global__ void __launch_bounds__(ALIGN_WARPS * 32) align_fwd_kernel(AlignArgs a
           int rF = __shfl_up_sync(FULL, sF, 1);
           int rC = __shfl_up_sync(FULL, sC, 1);
           if (lead) {
-            const uint32_t w = (jj < 2) ? cwc.x : cwc.y;
-            rC = int(((jj & 1) ? (w >> 16) : w) >> shift) & 0xff;
+            rC = code_of(cwc, jj, half, a.nib);
             const int2 tv = (jj == 0) ? c0 : (jj == 1) ? c1 : (jj == 2) ? c2 : c3;
             rH = tv.x;
             rF = tv.y;

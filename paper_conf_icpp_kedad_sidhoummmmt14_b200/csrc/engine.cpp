@@ -120,6 +120,7 @@ struct sw_handle_s {
   int64_t opt_bank_copy = 1;    // query-pair profile: second smem copy shifted by 64 B for odd lane groups
   int64_t opt_bank_skew = 1;    // mode-0 profile copies: per-copy bank skew (mode0_copies)
   int64_t opt_const_gaps = 1;   // gaps 10/2: the constant-gap kernel instantiations
+  int64_t opt_nibble = 1;       // alphabets <= 15: 4-bit DB stream
   int64_t opt_crit_min = CRIT_MIN_STEPS;                    // long-pair rule (see launch_all)
   int64_t opt_crit_pct = int64_t(CRIT_FRACTION * 100 + 0.5);
   int64_t opt_align_ws_mb = 2048;  // sw_align: traceback-code workspace per batch
@@ -142,6 +143,7 @@ struct sw_db_s {
   std::vector<int64_t> seq_len;  // caller order
   std::vector<int64_t> sorted_lens;  // descending, non-empty only (for overflow bounds)
   int n_long = 0;                // pairs [0, n_long) have len > T_LONG
+  int nib = 0;                   // 4-bit pair stream (alphabet <= 15)
   // per-DB constants of the pair table (computed once at load)
   double sum_short_len = 0, sum_long_len = 0, short_res = 0;
   int32_t max_short = 0, max_long = 0;
@@ -266,7 +268,7 @@ constexpr double SMALL_SEARCH_CELLS = 2e10;   // below this, minimise max(throug
 constexpr double CELLS_PER_CYCLE = 3500.0;    // whole-GPU throughput of the short-pair mode (config 3)
 
 static void choose_geom(const sw_handle_s* h, const std::vector<std::pair<int, int>>& slots, double Lavg, int& G,
-                        int& R, double Lmax = 0.0, double real_cells = 1e300) {
+                        int& R, double Lmax = 0.0, double real_cells = 1e300, bool nib = false) {
   if (h->opt_G > 0 && h->opt_R > 0) {
     G = int(h->opt_G);
     R = int(h->opt_R);
@@ -277,8 +279,10 @@ static void choose_geom(const sw_handle_s* h, const std::vector<std::pair<int, i
   double best = 1e300;
   G = 4;
   R = 24;
+  bool first = true;
   for (int g : Gs) {
     for (int r : Rs) {
+      if (nib && !short_config_supported(slots.empty() ? 0 : slots[0].second, g, r, true)) continue;
       // per-step overhead amortised over r rows; a lane of one sub-lane (r % 8 != 0)
       // has half the ILP.  The single-query kernel spills above 24 rows; the
       // query-pair kernel (its own register budget) does not lose at 32 (C3 A/B:
@@ -305,7 +309,7 @@ static void choose_geom(const sw_handle_s* h, const std::vector<std::pair<int, i
         const double cp = double(strips) * (Lmax + double(g * V)) * (18.4 * r + 99.0);
         cost = std::max(cost / CELLS_PER_CYCLE, cp);
       }
-      if (cost < best) { best = cost; G = g; R = r; }
+      if (cost < best || first) { best = cost; G = g; R = r; first = false; }
     }
   }
 }
@@ -365,6 +369,8 @@ int32_t sw_set_option(sw_handle_t h, const char* key, int64_t value) {
   } else if (k == "crit_pct") {
     if (value < 1) return set_err(h, SW_EINVAL, "crit_pct must be >= 1");
     h->opt_crit_pct = value;
+  } else if (k == "nibble") {
+    h->opt_nibble = value;
   } else if (k == "const_gaps") {
     h->opt_const_gaps = value;
   } else if (k == "query_pairs") {
@@ -397,7 +403,9 @@ int32_t sw_load_db(sw_handle_t h, const uint8_t* codes, const int64_t* offsets, 
     db->alpha = alphabet_size;
     Packed P;
     try {
-      pack_db(codes, offsets, n_seqs, alphabet_size, h->opt_t_long >= 0 ? h->opt_t_long : T_LONG, P);
+      // nucleotide-sized alphabets (<= 15 codes + PAD) get the 4-bit stream
+      pack_db(codes, offsets, n_seqs, alphabet_size, h->opt_t_long >= 0 ? h->opt_t_long : T_LONG, P,
+              h->opt_nibble != 0 && alphabet_size <= 15);
     } catch (const std::invalid_argument& e) {
       fail(SW_EINVAL, std::string("sw_load_db: ") + e.what());
     }
@@ -407,6 +415,7 @@ int32_t sw_load_db(sw_handle_t h, const uint8_t* codes, const int64_t* offsets, 
     db->n_res = P.n_res;
     db->max_len = P.max_len;
     db->n_long = P.n_long;
+    db->nib = P.nib;
     db->pairs = std::move(P.pairs);
     db->seq_len = std::move(P.seq_len);
     db->sorted_lens = std::move(P.sorted_lens);
@@ -571,10 +580,13 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
   double qsum = 0;
   for (int m : ms) qsum += m;
   int G1 = 4, R1 = 24, G0 = 4, R0 = 24;
-  if (!m1.empty()) choose_geom(h, m1, Lavg, G1, R1, double(db->max_short), qsum * double(db->n_res));
-  if (!m0.empty()) choose_geom(h, m0, Lavg, G0, R0, double(db->max_short), qsum * double(db->n_res));
-  if (!m1.empty() && !short_config_supported(1, G1, R1)) fail(SW_EUNSUPPORTED, "no query-pair kernel for this geometry");
-  if (!m0.empty() && !short_config_supported(0, G0, R0)) fail(SW_EUNSUPPORTED, "no single-query kernel for this geometry");
+  const bool nib = db->nib != 0;
+  if (!m1.empty()) choose_geom(h, m1, Lavg, G1, R1, double(db->max_short), qsum * double(db->n_res), nib);
+  if (!m0.empty()) choose_geom(h, m0, Lavg, G0, R0, double(db->max_short), qsum * double(db->n_res), nib);
+  if (!m1.empty() && !short_config_supported(1, G1, R1, nib))
+    fail(SW_EUNSUPPORTED, "no query-pair kernel for this geometry" + std::string(nib ? " (4-bit stream)" : ""));
+  if (!m0.empty() && !short_config_supported(0, G0, R0, nib))
+    fail(SW_EUNSUPPORTED, "no single-query kernel for this geometry" + std::string(nib ? " (4-bit stream)" : ""));
   const int NT = SCORE_NT, NG1 = NT / G1, NG0 = NT / G0, W = LONG_W;
   auto pairs_longer_than = [&](int64_t Lc) {  // pairs are sorted longest first
     int lo = 0, hi = np;
@@ -881,7 +893,7 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
   if (long_items > 0 && !combined) {
     int smem = smem_long;
     if (fork) smem = std::max(smem, 200 * 1024);  // SM-exclusive (see above)
-    const int occ = long_max_ctas_per_sm(smem);
+    const int occ = long_max_ctas_per_sm(smem, nib);
     if (occ <= 0) fail(SW_ECUDA, "long-pair kernel does not fit on an SM");
     const int grid = int(std::max<int64_t>(1, std::min<int64_t>(long_items, int64_t(occ) * h->sms)));
     SW_CK(h->wrap.ensure(size_t(grid) * al.wcap * sizeof(uint2)));
@@ -901,7 +913,7 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
     }
     std::pair<cudaEvent_t, cudaEvent_t>* ev = nullptr;
     record_begin(h, c.timing, 1, lst, ev);
-    SW_CK(launch_long(grid, smem, al, lst));
+    SW_CK(launch_long(grid, smem, al, lst, nib));
     if (ev) SW_CK(cudaEventRecord(ev->second, lst));
     if (fork) SW_CK(cudaEventRecord(h->ev_join, lst));
     ++out.launches;
@@ -935,7 +947,7 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
     const bool with_long = combined && mode == 0;
     if (with_long) smem = std::max(smem, smem_long);  // an item is short or long: the two uses share smem
     const bool cg = c.nGe == 0xfffefffeu && c.nGsGe == 0xfff4fff4u && h->opt_const_gaps != 0;
-    const int occ = with_long ? combined_max_ctas_per_sm(G, R, smem) : short_max_ctas_per_sm(mode, G, R, smem, cg);
+    const int occ = with_long ? combined_max_ctas_per_sm(G, R, smem, nib) : short_max_ctas_per_sm(mode, G, R, smem, cg, nib);
     if (occ <= 0) fail(SW_ECUDA, "short-pair kernel does not fit on an SM");
     const int64_t items = int64_t(n_short) + (with_long ? long_items : 0);
     const int grid = int(std::max<int64_t>(1, std::min<int64_t>(items, int64_t(occ) * h->sms)));
@@ -963,9 +975,9 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
     if (with_long) {
       SW_CK(h->wrap.ensure(size_t(grid) * al.wcap * sizeof(uint2)));
       al.wrap = h->wrap.as<uint2>();
-      SW_CK(launch_combined(G, R, grid, smem, as, al, c.st));
+      SW_CK(launch_combined(G, R, grid, smem, as, al, c.st, nib));
     } else {
-      SW_CK(launch_short(mode, G, R, grid, smem, as, c.st, cg));
+      SW_CK(launch_short(mode, G, R, grid, smem, as, c.st, cg, nib));
     }
     if (ev) SW_CK(cudaEventRecord(ev->second, c.st));
     ++out.launches;
@@ -1113,6 +1125,7 @@ int32_t sw_search(sw_handle_t h, const uint8_t* q_codes, const int64_t* q_offset
       r.qcodes = dq;
       r.qoff = h->qoff.as<int64_t>();
       r.stream = db->stream.as<uint16_t>();
+      r.nib = db->nib;
       r.pairs = db->dpairs.as<PairRec>();
       r.matrix = h->matrix.as<int8_t>();
       r.alpha = alpha;
@@ -1305,6 +1318,7 @@ int32_t sw_align(sw_handle_t h, const uint8_t* q_codes, const int64_t* q_offsets
       a.qcodes = h->a_qcodes.as<uint8_t>();
       a.qoff = h->a_qoff.as<int64_t>();
       a.stream = db->stream.as<uint16_t>();
+      a.nib = db->nib;
       a.pairs = db->dpairs.as<PairRec>();
       a.matrix = h->a_matrix.as<int8_t>();
       a.alpha = alpha;

@@ -185,8 +185,11 @@ __device__ __forceinline__ void wait_geq(const int* p, int need, int& seen, int 
 // above at rp[c] (c = column, rp = row base + G - 1), lane G-1 writes this
 // strip's bottom row at wp[t] (t = step).  LINKED (long items, G = 32): the
 // row above is produced concurrently by another warp of the CTA (Chain).
-template <int G, int R, bool LINKED, bool Q2 = false, int US = (Q2 ? 16 : ((R % 8 == 0) ? 8 : 4))>
-__device__ __forceinline__ void strip_pass(const uint8_t* sprof, int LS, int LB, const uint16_t* pstream, int L,
+// NIB: the pair's columns are bytes of two 4-bit codes (nucleotide DBs, SURVEY 8(f)
+// f4): lane 0 loads 4 columns per 32-bit word and spreads each byte into the
+// 16-bit pair word (two 8-bit codes) the rest of the pass uses.
+template <int G, int R, bool LINKED, bool Q2 = false, int US = (Q2 ? 16 : ((R % 8 == 0) ? 8 : 4)), bool NIB = false>
+__device__ __forceinline__ void strip_pass(const uint8_t* sprof, int LS, int LB, const void* pstream, int L,
                                            int T, int k, bool rd, bool wr, const uint2* __restrict__ rp,
                                            uint2* __restrict__ wp, const Chain& ch, uint32_t code_pad2,
                                            uint32_t nGe, uint32_t nGsGe, uint32_t& best, uint32_t shift = 0) {
@@ -199,7 +202,9 @@ __device__ __forceinline__ void strip_pass(const uint8_t* sprof, int LS, int LB,
   const uint32_t sbase = static_cast<uint32_t>(__cvta_generic_to_shared(sprof));
   uint32_t hdiag = 0, sH = 0, sF = 0, sC = code_pad2;
   const uint2* __restrict__ codes = reinterpret_cast<const uint2*>(pstream);
-  const uint32_t pad4 = code_pad2 | (code_pad2 << 16);
+  const uint32_t* __restrict__ codes4 = reinterpret_cast<const uint32_t*>(pstream);
+  const uint32_t pad4 = NIB ? ((code_pad2 & 0xfu) | ((code_pad2 >> 4) & 0xf0u)) * 0x01010101u
+                            : code_pad2 | (code_pad2 << 16);
   const uint32_t laneoff = uint32_t(k) * LB;
   const bool lead = (k == 0), tail = (k == G - 1);
   const uint2 z2 = make_uint2(0, 0);
@@ -214,7 +219,8 @@ __device__ __forceinline__ void strip_pass(const uint8_t* sprof, int LS, int LB,
   // lane 0 prefetch of block 0: 4 columns of codes and (if rd) 4 boundary cells.
   // L and t0 are multiples of 4, so one compare guards a whole block.
   auto load_block = [&](int t0, uint2& cw, uint2& b0, uint2& b1, uint2& b2, uint2& b3) {
-    cw = __ldcs(codes + (t0 >> 2));
+    if constexpr (NIB) cw = make_uint2(__ldcs(codes4 + (t0 >> 2)), 0u);
+    else cw = __ldcs(codes + (t0 >> 2));
     if (rd) {
       if constexpr (LINKED) {
         if (ch.in_ring) {
@@ -271,8 +277,13 @@ __device__ __forceinline__ void strip_pass(const uint8_t* sprof, int LS, int LB,
       uint32_t rF = __shfl_up_sync(FULL, sF, 1, G);
       uint32_t rC = __shfl_up_sync(FULL, sC, 1, G);
       if (lead) {
-        const uint32_t w = (j < 2) ? cwc.x : cwc.y;
-        rC = (j & 1) ? (w >> 16) : (w & 0xffffu);
+        if constexpr (NIB) {
+          const uint32_t b8 = (cwc.x >> (8 * j)) & 0xffu;
+          rC = (b8 & 0xfu) | ((b8 & 0xf0u) << 4);
+        } else {
+          const uint32_t w = (j < 2) ? cwc.x : cwc.y;
+          rC = (j & 1) ? (w >> 16) : (w & 0xffffu);
+        }
         const uint2 tv = (j == 0) ? c0 : (j == 1) ? c1 : (j == 2) ? c2 : c3;
         rH = tv.x;
         rF = tv.y;
@@ -364,7 +375,7 @@ __device__ __forceinline__ void stage_issue(ProfStage& ps, int b, int tag, const
 // CG: the gap penalties are the compile-time pair Gs = 10, Ge = 2 (BASELINE's
 // configuration): the cell update then encodes -Ge and -(Gs+Ge) as immediates,
 // one register operand fewer per VIADDMNMX / VIADD (register-file bandwidth).
-template <int G, int R, int NT, bool Q2, bool CG = false>
+template <int G, int R, int NT, bool Q2, bool CG = false, bool NIB = false>
 __device__ __forceinline__ void short_item(const ShortArgs& a, int item, uint8_t* smem, int& loaded, ProfStage& ps) {
   const uint32_t nGe = CG ? 0xfffefffeu : a.nGe, nGsGe = CG ? 0xfff4fff4u : a.nGsGe;
   uint8_t* sprof = smem;                         // the strip profile (bank-spread copies)
@@ -393,6 +404,8 @@ __device__ __forceinline__ void short_item(const ShortArgs& a, int item, uint8_t
     if (valid) pr = a.pairs[p];
     else { pr.off = 0; pr.len = 0; pr.id0 = -1; pr.id1 = -1; }
     if (Q2 && half && pr.id1 < 0) valid = false;  // odd leftover pair has no high half
+    const void* pstream = NIB ? static_cast<const void*>(reinterpret_cast<const uint8_t*>(a.stream) + pr.off)
+                              : static_cast<const void*>(a.stream + pr.off);
     int T = pr.len + G * SubLanes<R>::V;          // the last sub-lane finishes column len-1 at step T-2
     if (G < 32) T = __reduce_max_sync(FULL, T);   // warp-uniform trip count (shuffles)
     uint32_t best = 0;
@@ -430,7 +443,7 @@ __device__ __forceinline__ void short_item(const ShortArgs& a, int item, uint8_t
           }
           __syncwarp();
         }
-        strip_pass<G, R, false, true>(gprof, a.LS, a.LB, a.stream + pr.off, pr.len, T, k, rd, s + 1 < d.n_strips,
+        strip_pass<G, R, false, true, 16, NIB>(gprof, a.LS, a.LB, pstream, pr.len, T, k, rd, s + 1 < d.n_strips,
                                       bb, bb, Chain{}, a.code_pad2, nGe, nGsGe, best, half ? 8u : 0u);
         if (si.emit0 >= 0 || si.emit1 >= 0) {  // a query of either half ends with this strip
           uint32_t bg = best;
@@ -452,7 +465,8 @@ __device__ __forceinline__ void short_item(const ShortArgs& a, int item, uint8_t
           best &= (si.emit0 >= 0 ? 0xffff0000u : 0xffffffffu) & (si.emit1 >= 0 ? 0x0000ffffu : 0xffffffffu);
         }
       } else {
-        strip_pass<G, R, false>(gprof, a.LS, a.LB, a.stream + pr.off, pr.len, T, k, s > 0, s + 1 < d.n_strips,
+        strip_pass<G, R, false, false, ((R % 8 == 0) ? 8 : 4), NIB>(gprof, a.LS, a.LB, pstream, pr.len, T, k, s > 0,
+                                                                  s + 1 < d.n_strips,
                                 bb, bb, Chain{}, a.code_pad2, nGe, nGsGe, best);
       }
     }
@@ -489,6 +503,7 @@ struct LongShared {
   uint32_t best[LONG_W];
 };
 
+template <bool NIB>
 __device__ __forceinline__ void long_item(const LongArgs& a, int item, uint8_t* smem, LongShared& sh) {
   constexpr int W = LONG_W;
   // A producer may run LONG_RING - 4 steps ahead of its consumer's last published
@@ -557,7 +572,9 @@ __device__ __forceinline__ void long_item(const LongArgs& a, int item, uint8_t* 
         ch.grow_out = wrap;         // only reached when ns > W (P = 1): the round wrap
       }
       ch.out_prog = &s_prog[cbase + j];
-      strip_pass<32, LONG_R, true, false, LONG_US>(myprof, a.LSL, a.LBL, a.stream + pr.off, pr.len, T, lane, rd, wr,
+      const void* pstream = NIB ? static_cast<const void*>(reinterpret_cast<const uint8_t*>(a.stream) + pr.off)
+                                : static_cast<const void*>(a.stream + pr.off);
+      strip_pass<32, LONG_R, true, false, LONG_US, NIB>(myprof, a.LSL, a.LBL, pstream, pr.len, T, lane, rd, wr,
                                                    nullptr, nullptr, ch, a.code_pad2, a.nGe, a.nGsGe, best);
     }
 #pragma unroll
@@ -585,7 +602,7 @@ __device__ __forceinline__ void long_item(const LongArgs& a, int item, uint8_t* 
 // The short-pair kernel: one persistent launch per short-pair mode (query pairs,
 // single query), one (G, R) per launch, its own register budget (the query-pair
 // form keeps R = 32 rows per lane at 128 registers, 2 CTAs per SM).
-template <int G, int R, int NT, bool Q2, bool CG = false>
+template <int G, int R, int NT, bool Q2, bool CG = false, bool NIB = false>
 __global__ void __launch_bounds__(NT, 2) short_kernel(ShortArgs as) {
   extern __shared__ __align__(128) uint8_t smem[];
   __shared__ int s_item;
@@ -603,20 +620,21 @@ __global__ void __launch_bounds__(NT, 2) short_kernel(ShortArgs as) {
     const int item = s_item;
     __syncthreads();
     if (item >= as.n_items) break;
-    short_item<G, R, NT, Q2, CG>(as, item, smem, loaded, ps);
+    short_item<G, R, NT, Q2, CG, NIB>(as, item, smem, loaded, ps);
   }
 }
 
 // A long item as an out-of-line call: the combined single-query kernel below keeps
 // the short path's register allocation apart from it.
+template <bool NIB>
 __device__ __noinline__ void long_item_call(const LongArgs& a, int item, uint8_t* smem, LongShared& sh) {
-  long_item(a, item, smem, sh);
+  long_item<NIB>(a, item, smem, sh);
 }
 
 // Single-query searches with long pairs (C1/C2): ONE persistent launch, the long
 // items first (costliest), then the short items, so the longest pairs start at
 // once and the SMs that finish them move on to short items.
-template <int G, int R, int NT>
+template <int G, int R, int NT, bool NIB = false>
 __global__ void __launch_bounds__(NT, 2) combined_m0_kernel(ShortArgs as, LongArgs al) {
   extern __shared__ __align__(128) uint8_t smem[];
   __shared__ int s_item;
@@ -631,10 +649,10 @@ __global__ void __launch_bounds__(NT, 2) combined_m0_kernel(ShortArgs as, LongAr
     __syncthreads();
     if (item >= n_items) break;
     if (item < al.n_items) {
-      long_item_call(al, item, smem, sh);
+      long_item_call<NIB>(al, item, smem, sh);
       loaded = -1;  // the long item overwrote the strip profile
     } else {
-      short_item<G, R, NT, false>(as, item - al.n_items, smem, loaded, ps);
+      short_item<G, R, NT, false, false, NIB>(as, item - al.n_items, smem, loaded, ps);
     }
   }
 }
@@ -644,6 +662,7 @@ __global__ void __launch_bounds__(NT, 2) combined_m0_kernel(ShortArgs as, LongAr
 // on a side stream, one CTA per SM (a shared-memory request that leaves no room
 // for a short-pair CTA), so the co-resident short warps do not stretch the
 // critical path of the longest pairs.
+template <bool NIB>
 __global__ void __launch_bounds__(LONG_W * 32, 2) long_kernel(LongArgs al) {
   extern __shared__ __align__(128) uint8_t smem[];
   __shared__ int s_item;
@@ -654,7 +673,7 @@ __global__ void __launch_bounds__(LONG_W * 32, 2) long_kernel(LongArgs al) {
     const int item = s_item;
     __syncthreads();
     if (item >= al.n_items) break;
-    long_item(al, item, smem, sh);
+    long_item<NIB>(al, item, smem, sh);
   }
 }
 
@@ -670,8 +689,22 @@ typedef void (*short_fn)(ShortArgs);
 // constant-gap (Gs 10, Ge 2) instantiations of the geometries the cost model picks
 // for Swiss-Prot-like databases
 #define SW_CG_CASES(X) X(4, 32) X(4, 24) X(8, 32) X(8, 24) X(4, 16) X(8, 16)
+// 4-bit (nucleotide) database streams: a geometry subset (the cost model picks among them)
+#define SW_NIB_CASES(X) X(4, 16) X(4, 24) X(4, 32) X(8, 16) X(8, 24) X(16, 12) X(16, 24) X(32, 8) X(32, 16)
 
-static short_fn pick_short(int mode, int G, int R, bool cg = false) {
+static short_fn pick_short(int mode, int G, int R, bool cg = false, bool nib = false) {
+  if (nib) {
+    if (mode == 1) {
+#define X(g, r) if (G == g && R == r) return short_kernel<g, r, SCORE_NT, true, false, true>;
+      SW_NIB_CASES(X)
+#undef X
+    } else {
+#define X(g, r) if (G == g && R == r) return short_kernel<g, r, SCORE_NT, false, false, true>;
+      SW_NIB_CASES(X)
+#undef X
+    }
+    return nullptr;
+  }
   if (cg && mode == 1) {
 #define X(g, r) if (G == g && R == r) return short_kernel<g, r, SCORE_NT, true, true>;
     SW_CG_CASES(X)
@@ -694,7 +727,7 @@ static short_fn pick_short(int mode, int G, int R, bool cg = false) {
   return nullptr;
 }
 
-bool short_config_supported(int mode, int G, int R) { return pick_short(mode, G, R) != nullptr; }
+bool short_config_supported(int mode, int G, int R, bool nib) { return pick_short(mode, G, R, false, nib) != nullptr; }
 
 static int occupancy(const void* f, int threads, int smem_bytes) {
   if (smem_bytes > 48 * 1024) cudaFuncSetAttribute(f, cudaFuncAttributeMaxDynamicSharedMemorySize, smem_bytes);
@@ -703,16 +736,19 @@ static int occupancy(const void* f, int threads, int smem_bytes) {
   return n;
 }
 
-int short_max_ctas_per_sm(int mode, int G, int R, int smem_bytes, bool cg) {
-  short_fn f = pick_short(mode, G, R, cg);
-  if (!f) f = pick_short(mode, G, R);
+static short_fn pick_short_or_plain(int mode, int G, int R, bool cg, bool nib) {
+  short_fn f = pick_short(mode, G, R, cg && !nib, nib);
+  return (f || nib) ? f : pick_short(mode, G, R);
+}
+
+int short_max_ctas_per_sm(int mode, int G, int R, int smem_bytes, bool cg, bool nib) {
+  short_fn f = pick_short_or_plain(mode, G, R, cg, nib);
   return f ? occupancy(reinterpret_cast<const void*>(f), SCORE_NT, smem_bytes) : 0;
 }
 
 cudaError_t launch_short(int mode, int G, int R, int grid, int smem_bytes, const ShortArgs& a, cudaStream_t st,
-                         bool cg) {
-  short_fn f = pick_short(mode, G, R, cg);
-  if (!f) f = pick_short(mode, G, R);
+                         bool cg, bool nib) {
+  short_fn f = pick_short_or_plain(mode, G, R, cg, nib);
   if (!f) return cudaErrorInvalidValue;
   if (smem_bytes > 48 * 1024) {
     cudaError_t e = cudaFuncSetAttribute(f, cudaFuncAttributeMaxDynamicSharedMemorySize, smem_bytes);
@@ -723,21 +759,27 @@ cudaError_t launch_short(int mode, int G, int R, int grid, int smem_bytes, const
 }
 
 typedef void (*combined_fn)(ShortArgs, LongArgs);
-static combined_fn pick_combined(int G, int R) {
+static combined_fn pick_combined(int G, int R, bool nib) {
+  if (nib) {
+#define X(g, r) if (G == g && R == r) return combined_m0_kernel<g, r, SCORE_NT, true>;
+    SW_NIB_CASES(X)
+#undef X
+    return nullptr;
+  }
 #define X(g, r) if (G == g && R == r) return combined_m0_kernel<g, r, SCORE_NT>;
   SW_GEOM_CASES(X)
 #undef X
   return nullptr;
 }
 
-int combined_max_ctas_per_sm(int G, int R, int smem_bytes) {
-  combined_fn f = pick_combined(G, R);
+int combined_max_ctas_per_sm(int G, int R, int smem_bytes, bool nib) {
+  combined_fn f = pick_combined(G, R, nib);
   return f ? occupancy(reinterpret_cast<const void*>(f), SCORE_NT, smem_bytes) : 0;
 }
 
 cudaError_t launch_combined(int G, int R, int grid, int smem_bytes, const ShortArgs& as, const LongArgs& al,
-                            cudaStream_t st) {
-  combined_fn f = pick_combined(G, R);
+                            cudaStream_t st, bool nib) {
+  combined_fn f = pick_combined(G, R, nib);
   if (!f) return cudaErrorInvalidValue;
   if (smem_bytes > 48 * 1024) {
     cudaError_t e = cudaFuncSetAttribute(f, cudaFuncAttributeMaxDynamicSharedMemorySize, smem_bytes);
@@ -747,16 +789,18 @@ cudaError_t launch_combined(int G, int R, int grid, int smem_bytes, const ShortA
   return cudaGetLastError();
 }
 
-int long_max_ctas_per_sm(int smem_bytes) {
-  return occupancy(reinterpret_cast<const void*>(long_kernel), LONG_W * 32, smem_bytes);
+int long_max_ctas_per_sm(int smem_bytes, bool nib) {
+  return occupancy(nib ? reinterpret_cast<const void*>(long_kernel<true>) : reinterpret_cast<const void*>(long_kernel<false>),
+                   LONG_W * 32, smem_bytes);
 }
 
-cudaError_t launch_long(int grid, int smem_bytes, const LongArgs& a, cudaStream_t st) {
+cudaError_t launch_long(int grid, int smem_bytes, const LongArgs& a, cudaStream_t st, bool nib) {
+  auto f = nib ? long_kernel<true> : long_kernel<false>;
   if (smem_bytes > 48 * 1024) {
-    cudaError_t e = cudaFuncSetAttribute(long_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize, smem_bytes);
+    cudaError_t e = cudaFuncSetAttribute(f, cudaFuncAttributeMaxDynamicSharedMemorySize, smem_bytes);
     if (e != cudaSuccess) return e;
   }
-  long_kernel<<<grid, LONG_W * 32, smem_bytes, st>>>(a);
+  f<<<grid, LONG_W * 32, smem_bytes, st>>>(a);
   return cudaGetLastError();
 }
 
@@ -816,11 +860,10 @@ __global__ void __launch_bounds__(RESCORE_WARPS * 32) rescore_kernel(RescoreArgs
     const uint8_t* qc = a.qcodes + a.qoff[o.q];
     const int m = int(a.qoff[o.q + 1] - a.qoff[o.q]);
     const int L = pr.len;
-    const uint32_t shift = o.half ? 8u : 0u;
+    const int half = o.half;
     const int nstrips = (m + 32 * R - 1) / (32 * R);
     const int T = L + 32;
-    const uint2* __restrict__ codes = reinterpret_cast<const uint2*>(a.stream + pr.off);
-    const uint32_t padw = uint32_t(pad) * 0x01010101u;
+    const uint2 padw = pad_codes4(pad, a.nib);
     const int blk = e % a.ne_slots;
     int2* grow = a.grows + (int64_t)blk * K * a.bcap;
     unsigned long long* gflag = a.gflags + (int64_t)blk * K;
@@ -871,11 +914,11 @@ __global__ void __launch_bounds__(RESCORE_WARPS * 32) rescore_kernel(RescoreArgs
       }
       int hdiag = 0, sH = 0, sF = 0, sC = pad;
       const int2 z2 = make_int2(0, 0);
-      uint2 cw = make_uint2(padw, padw);
+      uint2 cw = padw;
       int2 tb0 = z2, tb1 = z2, tb2 = z2, tb3 = z2;
       if (rd && L > 0) wait_in(in_base + min(4 + 31 + RESCORE_LAG, L + 32));
       if (lead && L > 0) {
-        cw = codes[0];
+        cw = load_codes4(a.stream, pr.off, 0, a.nib);
         if (rd) { tb0 = __ldcg(rp + 0); tb1 = __ldcg(rp + 1); tb2 = __ldcg(rp + 2); tb3 = __ldcg(rp + 3); }
       }
       __syncwarp();
@@ -885,12 +928,12 @@ __global__ void __launch_bounds__(RESCORE_WARPS * 32) rescore_kernel(RescoreArgs
         if (rd && t0 + 4 < L) wait_in(in_base + min(t0 + 8 + 31 + RESCORE_LAG, L + 32));
         if (lead) {
           if (t0 + 4 < L) {
-            cw = codes[(t0 + 4) >> 2];
+            cw = load_codes4(a.stream, pr.off, t0 + 4, a.nib);
             if (rd) {
               tb0 = __ldcg(rp + t0 + 4); tb1 = __ldcg(rp + t0 + 5); tb2 = __ldcg(rp + t0 + 6); tb3 = __ldcg(rp + t0 + 7);
             }
           } else {
-            cw = make_uint2(padw, padw);
+            cw = padw;
             tb0 = z2; tb1 = z2; tb2 = z2; tb3 = z2;
           }
         }
@@ -901,8 +944,7 @@ __global__ void __launch_bounds__(RESCORE_WARPS * 32) rescore_kernel(RescoreArgs
           int rF = __shfl_up_sync(FULL, sF, 1);
           int rC = __shfl_up_sync(FULL, sC, 1);
           if (lead) {
-            const uint32_t w = (jj < 2) ? cwc.x : cwc.y;
-            rC = int(((jj & 1) ? (w >> 16) : w) >> shift) & 0xff;
+            rC = code_of(cwc, jj, half, a.nib);
             const int2 tv = (jj == 0) ? c0 : (jj == 1) ? c1 : (jj == 2) ? c2 : c3;
             rH = tv.x;
             rF = tv.y;

@@ -25,7 +25,8 @@ namespace swdual {
 
 static unsigned n_threads() { return std::max(1u, std::min(16u, std::thread::hardware_concurrency())); }
 
-void pack_db(const uint8_t* codes, const int64_t* offsets, int64_t n_seqs, int alpha, int64_t t_long, Packed& P) {
+void pack_db(const uint8_t* codes, const int64_t* offsets, int64_t n_seqs, int alpha, int64_t t_long, Packed& P,
+             bool nib) {
   if (n_seqs < 0) throw std::invalid_argument("n_seqs < 0");
   if (alpha < 1 || alpha > 32) throw std::invalid_argument("alphabet_size must be in 1..32");
   if (n_seqs > 0 && !offsets) throw std::invalid_argument("offsets is NULL");
@@ -78,6 +79,33 @@ void pack_db(const uint8_t* codes, const int64_t* offsets, int64_t n_seqs, int a
     r.pad_ = 0;
     off += r.len;
     if (L > t_long) P.n_long = int(p + 1);
+  }
+  if (nib && alpha > 15) throw std::invalid_argument("4-bit codes need alphabet_size <= 15");
+  P.nib = nib ? 1 : 0;
+  if (nib) {  // one byte per pair column: two 4-bit codes (PAD = alpha <= 15)
+    P.stream.assign(size_t(std::max<int64_t>((off + 1) / 2, 4)), 0);
+    uint8_t* bytes = reinterpret_cast<uint8_t*>(P.stream.data());
+    std::fill(bytes, bytes + 2 * P.stream.size(), uint8_t(alpha | (alpha << 4)));
+    const unsigned nt = n_threads();
+    std::vector<std::thread> th;
+    for (unsigned t = 0; t < nt; ++t)
+      th.emplace_back([&, t] {
+        for (size_t p = t; p < np; p += nt) {
+          const PairRec& r = P.pairs[p];
+          const uint8_t* s0 = codes + offsets[r.id0];
+          const int64_t l0 = P.seq_len[size_t(r.id0)];
+          const uint8_t* s1 = r.id1 >= 0 ? codes + offsets[r.id1] : nullptr;
+          const int64_t l1 = r.id1 >= 0 ? P.seq_len[size_t(r.id1)] : 0;
+          uint8_t* w = bytes + r.off;
+          for (int64_t c = 0; c < r.len; ++c) {
+            const uint8_t a = c < l0 ? s0[c] : uint8_t(alpha);
+            const uint8_t b = c < l1 ? s1[c] : uint8_t(alpha);
+            w[c] = uint8_t(a | (b << 4));
+          }
+        }
+      });
+    for (auto& x : th) x.join();
+    return;
   }
   P.stream.assign(size_t(std::max<int64_t>(off, 4)), uint16_t(alpha | (alpha << 8)));
   const uint16_t pad = uint16_t(alpha);

@@ -253,6 +253,24 @@ __device__ __forceinline__ void fence_proxy_async_smem() {
   asm volatile("fence.proxy.async.shared::cta;" ::: "memory");
 }
 
+// Pair-stream access of the int32 paths (re-score, sw_align): 4 columns per load,
+// either 16-bit columns (uint2) or, for 4-bit nucleotide streams, bytes (uint32).
+__device__ __forceinline__ uint2 load_codes4(const uint16_t* stream, int64_t off, int t0, int nib) {
+  if (nib) return make_uint2(reinterpret_cast<const uint32_t*>(reinterpret_cast<const uint8_t*>(stream) + off)[t0 >> 2], 0u);
+  return reinterpret_cast<const uint2*>(stream + off)[t0 >> 2];
+}
+// the letter of column jj (0..3) of a 4-column block, half 0 (id0) or 1 (id1)
+__device__ __forceinline__ int code_of(uint2 cw, int jj, int half, int nib) {
+  if (nib) return int((cw.x >> (8 * jj + 4 * half)) & 0xfu);
+  const uint32_t w = (jj < 2) ? cw.x : cw.y;
+  return int((((jj & 1) ? (w >> 16) : w) >> (8 * half)) & 0xffu);
+}
+__device__ __forceinline__ uint2 pad_codes4(int pad, int nib) {
+  const uint32_t b = nib ? uint32_t(pad | (pad << 4)) : uint32_t(pad);
+  const uint32_t w = b * 0x01010101u;
+  return make_uint2(w, nib ? 0u : w);
+}
+
 // GPU-scope counters (sw_align's CTA-to-CTA chains of very tall pairs).
 __device__ __forceinline__ int ld_acquire_gpu(const int* p) {
   int v;

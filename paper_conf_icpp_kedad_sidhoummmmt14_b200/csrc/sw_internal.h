@@ -18,16 +18,21 @@ struct PairRec {
   int32_t pad_;
 };
 
-// Host-packed database (packer.cpp).
+// Host-packed database (packer.cpp).  nib = 0: 16-bit pair columns (8-bit codes,
+// protein); nib = 1 (alphabet <= 15, nucleotides): 8-bit pair
+// columns of two 4-bit codes (low nibble id0, high nibble id1), stored as bytes
+// in `stream`; pair p's column c is byte off + c.
 struct Packed {
   std::vector<PairRec> pairs;        // sorted longest first
-  std::vector<uint16_t> stream;      // interleaved pair columns
+  std::vector<uint16_t> stream;      // interleaved pair columns (bytes when nib)
+  int nib = 0;
   std::vector<int64_t> seq_len;      // caller order
   std::vector<int64_t> sorted_lens;  // non-empty lengths, descending
   int64_t n_res = 0, max_len = 0;
   int n_long = 0;                    // pairs [0, n_long) are longer than t_long
 };
-void pack_db(const uint8_t* codes, const int64_t* offsets, int64_t n_seqs, int alpha, int64_t t_long, Packed& P);
+void pack_db(const uint8_t* codes, const int64_t* offsets, int64_t n_seqs, int alpha, int64_t t_long, Packed& P,
+             bool nib = false);
 
 // A pair whose int16 maximum reached the overflow threshold:
 // re-scored exactly in int32.
@@ -145,6 +150,7 @@ struct RescoreArgs {
   const uint8_t* qcodes;     // all queries, concatenated
   const int64_t* qoff;       // [nq+1]
   const uint16_t* stream;
+  int nib;                   // 4-bit pair columns (bytes) instead of 16-bit
   const PairRec* pairs;
   const int8_t* matrix;      // alpha x alpha
   int alpha;
@@ -184,17 +190,18 @@ cudaError_t launch_build_profile_q2(const uint8_t* qa, int ma, const uint8_t* qb
 // per launch.  Long-pair kernel: LONG_W chained warps per CTA.
 constexpr int SCORE_NT = 256;       // threads per CTA of both
 constexpr int LONG_W = SCORE_NT / 32;
-bool short_config_supported(int mode, int G, int R);
-// cg: the gaps are Gs = 10, Ge = 2 -- use the constant-gap instantiation when one exists
-int short_max_ctas_per_sm(int mode, int G, int R, int smem_bytes, bool cg = false);
+// cg: the gaps are Gs = 10, Ge = 2 -- use the constant-gap instantiation when one exists;
+// nib: the DB stream holds 4-bit codes (only the SW_NIB_CASES geometries exist)
+bool short_config_supported(int mode, int G, int R, bool nib = false);
+int short_max_ctas_per_sm(int mode, int G, int R, int smem_bytes, bool cg = false, bool nib = false);
 cudaError_t launch_short(int mode, int G, int R, int grid, int smem_bytes, const ShortArgs& a, cudaStream_t st,
-                         bool cg = false);
-int long_max_ctas_per_sm(int smem_bytes);
+                         bool cg = false, bool nib = false);
+int long_max_ctas_per_sm(int smem_bytes, bool nib = false);
+cudaError_t launch_long(int grid, int smem_bytes, const LongArgs& a, cudaStream_t st, bool nib = false);
 // single-query searches with long pairs: long items and mode-0 short items in one launch
-int combined_max_ctas_per_sm(int G, int R, int smem_bytes);
+int combined_max_ctas_per_sm(int G, int R, int smem_bytes, bool nib = false);
 cudaError_t launch_combined(int G, int R, int grid, int smem_bytes, const ShortArgs& as, const LongArgs& al,
-                            cudaStream_t st);
-cudaError_t launch_long(int grid, int smem_bytes, const LongArgs& a, cudaStream_t st);
+                            cudaStream_t st, bool nib = false);
 cudaError_t launch_rescore(int grid, const RescoreArgs& a, cudaStream_t st);
 // scores[q * stride + cols[c]] = 0 for every query q < nq and column c < ncols
 cudaError_t launch_zero_columns(int32_t* scores, int64_t stride, int nq, const int64_t* cols, int64_t ncols,
@@ -224,6 +231,7 @@ struct AlignArgs {
   const uint8_t* qcodes;     // all queries, concatenated
   const int64_t* qoff;       // [nq+1]
   const uint16_t* stream;
+  int nib;                   // 4-bit pair columns (bytes) instead of 16-bit
   const PairRec* pairs;
   const int8_t* matrix;      // alpha x alpha
   int alpha;

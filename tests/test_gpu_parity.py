@@ -477,3 +477,36 @@ def test_constant_gap_kernels(cg, pairs):
     qc, qo = _seqs([700, 129, 64, 3100, 2], rng)
     got = gpu_scores(qc, qo, dc, do, opts={"const_gaps": cg, "query_pairs": pairs})
     np.testing.assert_array_equal(got, oracle_scores(qc, qo, dc, do))
+
+
+NIB_GEOMS = [(4, 16), (4, 24), (4, 32), (8, 16), (8, 24), (16, 12), (16, 24), (32, 8), (32, 16)]
+
+
+@pytest.mark.parametrize("G,R", NIB_GEOMS)
+@pytest.mark.parametrize("pairs", [0, 1])
+def test_nibble_stream_geometries(G, R, pairs):
+    """alphabets <= 15 (DNA/RNA, alphabet 5 with N) are packed 4 bits
+    per residue (two codes per byte of the pair stream, half the DB bytes); every
+    4-bit instantiation, both query modes, multi-strip queries and PAD columns."""
+    sw = _pkg()
+    rng = np.random.default_rng(200 + G * 3 + R + pairs)
+    S = sw.nucleotide_matrix(2, -3)
+    dc, do = _seqs(list(rng.integers(1, 600, size=130)) + [0, 1, 2, 5], rng, alpha=5)
+    qc, qo = _seqs([3 * G * R + 7, G * R, 40, 1, 333], rng, alpha=5)
+    got = gpu_scores(qc, qo, dc, do, S=S, gs=5, ge=2, alpha=5,
+                     opts={"force_G": G, "force_R": R, "query_pairs": pairs})
+    np.testing.assert_array_equal(got, oracle_scores(qc, qo, dc, do, S=S.astype(np.int32), gs=5, ge=2))
+
+
+@pytest.mark.parametrize("opts", [{"t_long": 64}, {"overflow_threshold": 30}, {"nibble": 0}, {}])
+def test_nibble_stream_long_rescore_and_off(opts):
+    """4-bit streams through the intra-task kernel (forced long pairs, queries of
+    1 to 26 strips), the int32 re-score (forced threshold), and the 8-bit layout
+    (option nibble 0) for the same nucleotide DB: all equal to the oracle."""
+    sw = _pkg()
+    rng = np.random.default_rng(210 + len(str(opts)))
+    S = sw.nucleotide_matrix(1, -1)
+    dc, do = _seqs(list(rng.integers(1, 900, size=80)) + [0, 1, 66, 67], rng, alpha=5)
+    qc, qo = _seqs([1, 100, 513, 2400, 4100, 13000], rng, alpha=5)
+    got = gpu_scores(qc, qo, dc, do, S=S, gs=0, ge=2, alpha=5, opts=opts)
+    np.testing.assert_array_equal(got, oracle_scores(qc, qo, dc, do, S=S.astype(np.int32), gs=0, ge=2))

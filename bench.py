@@ -420,16 +420,18 @@ def run_ours(args):
         cpu = cpu_baseline(c, args.cpu_baseline_cells)
 
     # second denominator: the measured register-resident cell-update
-    # microbenchmark at the kernel's occupancy (tools/dpx_microbench.cu, 2 CTAs/SM)
+    # ceiling of the query-pair kernel's shape (tools/dpx_microbench2.cu: R = 32 rows,
+    # 2 chains, 256 threads x 2 CTAs/SM, penalties as immediates)
     micro = None
-    mpath = os.path.join(ROOT, "profiles", "r01_dpx_microbench.jsonl")
+    mpath = os.path.join(ROOT, "profiles", "r02_dpx_microbench2.jsonl")
     if os.path.exists(mpath):
         for ln in open(mpath):
             try:
                 d = json.loads(ln)
             except ValueError:
                 continue
-            if d.get("probe") == "gotoh_cellpair_D_max3_R24" and d.get("blocks_per_sm") == 2:
+            if (d.get("R"), d.get("chains"), d.get("lds"), d.get("xch"), d.get("threads"),
+                    d.get("ctas_per_sm")) == (32, 2, 0, 0, 256, 2) and "GCUPS" in d:
                 micro = float(d["GCUPS"])
     if rank == 0:
         line = {"metric": METRIC, "value": round(value, 2), "unit": "GCUPS", "n_gpus": world, "steps": args.steps,
@@ -450,8 +452,9 @@ def run_ours(args):
                                            f"derived from unit counts + measured pipe attribution)",
                              "microbench_ceiling": micro,
                              "frac_vs_microbench": round(achieved / micro, 4) if (achieved and micro) else None,
-                             "microbench_basis": "register-resident s16x2 cell update, same 3.5-ALU-op form, 2 CTAs/SM, "
-                                                 "no memory or shuffles (profiles/r01_dpx_microbench.jsonl)"},
+                             "microbench_basis": "register-resident s16x2 cell update, same 3.5-ALU-op form, R = 32 rows "
+                                                 "x 2 chains, 2 CTAs/SM, no memory or shuffles "
+                                                 "(profiles/r02_dpx_microbench2.jsonl)"},
                 "cpu_baseline": cpu, "e2e": e2e, "gpu_launches": int(nl_sum * args.steps),
                 **({"verified_sample": args.verify, "verified": verified} if args.verify else {}),
                 "clocks": clk,

@@ -121,6 +121,7 @@ struct sw_handle_s {
   int64_t opt_bank_skew = 1;    // mode-0 profile copies: per-copy bank skew (mode0_copies)
   int64_t opt_const_gaps = 1;   // gaps 10/2: the constant-gap kernel instantiations
   int64_t opt_nibble = 1;       // alphabets <= 15: 4-bit DB stream
+  int64_t opt_small_ctas = 1;   // latency-bound single-query searches: 32-thread CTAs
   int64_t opt_crit_min = CRIT_MIN_STEPS;                    // long-pair rule (see launch_all)
   int64_t opt_crit_pct = int64_t(CRIT_FRACTION * 100 + 0.5);
   int64_t opt_align_ws_mb = 2048;  // sw_align: traceback-code workspace per batch
@@ -265,6 +266,7 @@ static ProfGeom make_geom(int G, int R, int m, int alpha, bool long_mode = false
 // of shuffles / loads (fit on config 1: G,R = 4,24 / 8,24 / 16,16 / 16,8 / 32,8 /
 // 32,12 measured 1.11 / 0.60 / 0.39 / 0.45 / 0.26 / 0.38 ms, model within 12 %).
 constexpr double SMALL_SEARCH_CELLS = 2e10;   // below this, minimise max(throughput, critical path)
+constexpr double SMALL_LATENCY_CELLS = 1e9;   // below this, 32-lane groups get their own 32-thread CTAs
 constexpr double CELLS_PER_CYCLE = 3500.0;    // whole-GPU throughput of the short-pair mode (config 3)
 
 static void choose_geom(const sw_handle_s* h, const std::vector<std::pair<int, int>>& slots, double Lavg, int& G,
@@ -369,6 +371,8 @@ int32_t sw_set_option(sw_handle_t h, const char* key, int64_t value) {
   } else if (k == "crit_pct") {
     if (value < 1) return set_err(h, SW_EINVAL, "crit_pct must be >= 1");
     h->opt_crit_pct = value;
+  } else if (k == "small_ctas") {
+    h->opt_small_ctas = value;
   } else if (k == "nibble") {
     h->opt_nibble = value;
   } else if (k == "const_gaps") {
@@ -587,7 +591,14 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
     fail(SW_EUNSUPPORTED, "no query-pair kernel for this geometry" + std::string(nib ? " (4-bit stream)" : ""));
   if (!m0.empty() && !short_config_supported(0, G0, R0, nib))
     fail(SW_EUNSUPPORTED, "no single-query kernel for this geometry" + std::string(nib ? " (4-bit stream)" : ""));
-  const int NT = SCORE_NT, NG1 = NT / G1, NG0 = NT / G0, W = LONG_W;
+  // Latency-bound single-query searches (C1-sized) with 32-lane groups run one
+  // lane group per 32-thread CTA: the groups then spread over all SMs instead of
+  // eight per CTA sharing one SM's ALU pipe, which shortens the critical path.
+  const bool small_ctas = !m0.empty() && G0 == 32 && qsum * double(db->n_res) < SMALL_LATENCY_CELLS &&
+                          h->opt_small_ctas != 0 && short_config_supported(0, G0, R0, nib, 32);
+  int NT0 = SCORE_NT;
+  const int NT1 = SCORE_NT, NG1 = NT1 / G1, W = LONG_W;
+  int NG0 = NT0 / G0;
   auto pairs_longer_than = [&](int64_t Lc) {  // pairs are sorted longest first
     int lo = 0, hi = np;
     while (lo < hi) { const int mid = (lo + hi) / 2; if (db->pairs[size_t(mid)].len > Lc) lo = mid + 1; else hi = mid; }
@@ -704,6 +715,10 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
     if (sl.nlong > 0) any_long = true;
   }
   const bool combined = any_long && any_m0 && !any_q2;
+  if (small_ctas && !combined) {  // (a combined launch needs whole CTAs for its long items)
+    NT0 = 32;
+    NG0 = NT0 / G0;
+  }
   // ---- long work: one item per (query, long pair), or per `pack` pairs
   std::vector<LongQuery> ldesc;
   struct LItem { double cost; int q, it; };
@@ -947,7 +962,9 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
     const bool with_long = combined && mode == 0;
     if (with_long) smem = std::max(smem, smem_long);  // an item is short or long: the two uses share smem
     const bool cg = c.nGe == 0xfffefffeu && c.nGsGe == 0xfff4fff4u && h->opt_const_gaps != 0;
-    const int occ = with_long ? combined_max_ctas_per_sm(G, R, smem, nib) : short_max_ctas_per_sm(mode, G, R, smem, cg, nib);
+    const int nt = mode == 1 ? NT1 : NT0;
+    const int occ = with_long ? combined_max_ctas_per_sm(G, R, smem, nib)
+                              : short_max_ctas_per_sm(mode, G, R, smem, cg, nib, nt);
     if (occ <= 0) fail(SW_ECUDA, "short-pair kernel does not fit on an SM");
     const int64_t items = int64_t(n_short) + (with_long ? long_items : 0);
     const int grid = int(std::max<int64_t>(1, std::min<int64_t>(items, int64_t(occ) * h->sms)));
@@ -955,6 +972,7 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
     const int32_t max_short = min_pb < np ? db->pairs[size_t(min_pb)].len : 0;
     as.bcap = ((max_short + 4 * G + 8 + 4) + 3) / 4 * 4;  // wave width up to V*G sub-lanes + align pad
     DevBuf& bbuf = mode == 1 ? h->bbuf1 : h->bbuf0;
+    const int NT = mode == 1 ? NT1 : NT0;
     if (max_strips > 1) SW_CK(bbuf.ensure(size_t(grid) * (NT / G) * as.bcap * sizeof(uint2)));
     as.bbuf = max_strips > 1 ? bbuf.as<uint2>() : nullptr;
     as.stream = db->stream.as<uint16_t>();
@@ -977,7 +995,7 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
       al.wrap = h->wrap.as<uint2>();
       SW_CK(launch_combined(G, R, grid, smem, as, al, c.st, nib));
     } else {
-      SW_CK(launch_short(mode, G, R, grid, smem, as, c.st, cg, nib));
+      SW_CK(launch_short(mode, G, R, grid, smem, as, c.st, cg, nib, nt));
     }
     if (ev) SW_CK(cudaEventRecord(ev->second, c.st));
     ++out.launches;

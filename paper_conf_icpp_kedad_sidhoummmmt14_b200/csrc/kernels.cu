@@ -692,7 +692,17 @@ typedef void (*short_fn)(ShortArgs);
 // 4-bit (nucleotide) database streams: a geometry subset (the cost model picks among them)
 #define SW_NIB_CASES(X) X(4, 16) X(4, 24) X(4, 32) X(8, 16) X(8, 24) X(16, 12) X(16, 24) X(32, 8) X(32, 16)
 
-static short_fn pick_short(int mode, int G, int R, bool cg = false, bool nib = false) {
+// one-group CTAs for latency-bound single-query searches
+#define SW_SMALL_CASES(X) X(32, 8) X(32, 12) X(32, 16)
+
+static short_fn pick_short(int mode, int G, int R, bool cg = false, bool nib = false, int nt = SCORE_NT) {
+  if (nt == 32) {
+    if (mode != 0 || nib) return nullptr;
+#define X(g, r) if (G == g && R == r) return short_kernel<g, r, 32, false>;
+    SW_SMALL_CASES(X)
+#undef X
+    return nullptr;
+  }
   if (nib) {
     if (mode == 1) {
 #define X(g, r) if (G == g && R == r) return short_kernel<g, r, SCORE_NT, true, false, true>;
@@ -727,7 +737,9 @@ static short_fn pick_short(int mode, int G, int R, bool cg = false, bool nib = f
   return nullptr;
 }
 
-bool short_config_supported(int mode, int G, int R, bool nib) { return pick_short(mode, G, R, false, nib) != nullptr; }
+bool short_config_supported(int mode, int G, int R, bool nib, int nt) {
+  return pick_short(mode, G, R, false, nib, nt) != nullptr;
+}
 
 static int occupancy(const void* f, int threads, int smem_bytes) {
   if (smem_bytes > 48 * 1024) cudaFuncSetAttribute(f, cudaFuncAttributeMaxDynamicSharedMemorySize, smem_bytes);
@@ -736,25 +748,26 @@ static int occupancy(const void* f, int threads, int smem_bytes) {
   return n;
 }
 
-static short_fn pick_short_or_plain(int mode, int G, int R, bool cg, bool nib) {
+static short_fn pick_short_or_plain(int mode, int G, int R, bool cg, bool nib, int nt) {
+  if (nt != SCORE_NT) return pick_short(mode, G, R, false, nib, nt);
   short_fn f = pick_short(mode, G, R, cg && !nib, nib);
   return (f || nib) ? f : pick_short(mode, G, R);
 }
 
-int short_max_ctas_per_sm(int mode, int G, int R, int smem_bytes, bool cg, bool nib) {
-  short_fn f = pick_short_or_plain(mode, G, R, cg, nib);
-  return f ? occupancy(reinterpret_cast<const void*>(f), SCORE_NT, smem_bytes) : 0;
+int short_max_ctas_per_sm(int mode, int G, int R, int smem_bytes, bool cg, bool nib, int nt) {
+  short_fn f = pick_short_or_plain(mode, G, R, cg, nib, nt);
+  return f ? occupancy(reinterpret_cast<const void*>(f), nt, smem_bytes) : 0;
 }
 
 cudaError_t launch_short(int mode, int G, int R, int grid, int smem_bytes, const ShortArgs& a, cudaStream_t st,
-                         bool cg, bool nib) {
-  short_fn f = pick_short_or_plain(mode, G, R, cg, nib);
+                         bool cg, bool nib, int nt) {
+  short_fn f = pick_short_or_plain(mode, G, R, cg, nib, nt);
   if (!f) return cudaErrorInvalidValue;
   if (smem_bytes > 48 * 1024) {
     cudaError_t e = cudaFuncSetAttribute(f, cudaFuncAttributeMaxDynamicSharedMemorySize, smem_bytes);
     if (e != cudaSuccess) return e;
   }
-  f<<<grid, SCORE_NT, smem_bytes, st>>>(a);
+  f<<<grid, nt, smem_bytes, st>>>(a);
   return cudaGetLastError();
 }
 

@@ -192,10 +192,12 @@ constexpr int SCORE_NT = 256;       // threads per CTA of both
 constexpr int LONG_W = SCORE_NT / 32;
 // cg: the gaps are Gs = 10, Ge = 2 -- use the constant-gap instantiation when one exists;
 // nib: the DB stream holds 4-bit codes (only the SW_NIB_CASES geometries exist)
-bool short_config_supported(int mode, int G, int R, bool nib = false);
-int short_max_ctas_per_sm(int mode, int G, int R, int smem_bytes, bool cg = false, bool nib = false);
+// nt: threads per CTA (SCORE_NT, or 32 for latency-bound single-query searches at G = 32)
+bool short_config_supported(int mode, int G, int R, bool nib = false, int nt = SCORE_NT);
+int short_max_ctas_per_sm(int mode, int G, int R, int smem_bytes, bool cg = false, bool nib = false,
+                          int nt = SCORE_NT);
 cudaError_t launch_short(int mode, int G, int R, int grid, int smem_bytes, const ShortArgs& a, cudaStream_t st,
-                         bool cg = false, bool nib = false);
+                         bool cg = false, bool nib = false, int nt = SCORE_NT);
 int long_max_ctas_per_sm(int smem_bytes, bool nib = false);
 cudaError_t launch_long(int grid, int smem_bytes, const LongArgs& a, cudaStream_t st, bool nib = false);
 // single-query searches with long pairs: long items and mode-0 short items in one launch

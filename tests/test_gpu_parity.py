@@ -510,3 +510,16 @@ def test_nibble_stream_long_rescore_and_off(opts):
     qc, qo = _seqs([1, 100, 513, 2400, 4100, 13000], rng, alpha=5)
     got = gpu_scores(qc, qo, dc, do, S=S, gs=0, ge=2, alpha=5, opts=opts)
     np.testing.assert_array_equal(got, oracle_scores(qc, qo, dc, do, S=S.astype(np.int32), gs=0, ge=2))
+
+
+@pytest.mark.parametrize("small", [0, 1])
+def test_small_search_one_group_ctas(small):
+    """Latency-bound single-query searches at G = 32 run one lane group per
+    32-thread CTA (option small_ctas); both layouts equal the oracle, including
+    multi-strip queries and the longest pair setting the critical path."""
+    rng = np.random.default_rng(230 + small)
+    dc, do = _seqs(list(rng.integers(1, 700, size=300)) + [2005, 0, 1], rng)
+    for ql in ([144], [700], [33]):
+        qc, qo = _seqs(ql, rng)
+        got = gpu_scores(qc, qo, dc, do, opts={"small_ctas": small})
+        np.testing.assert_array_equal(got, oracle_scores(qc, qo, dc, do))

@@ -320,6 +320,17 @@ int32_t sw_pack_db_host(const uint8_t* codes, const int64_t* offsets, int64_t n_
                         int64_t t_long, sw_pair_t* pairs, int64_t* n_pairs, uint16_t* stream,
                         int64_t* stream_words, int64_t* n_long);
 
+/*
+ * Host-only gather of selected sequences (the multi-GPU layer's shard cut, SURVEY
+ * 8(a) a3): sequences ids[0..n_ids) of (codes, offsets[n_seqs + 1]) are copied, in
+ * that order, to out_codes with out_offsets[n_ids + 1] (starting at 0).  Two-phase:
+ * with out_codes == NULL only *n_out (residues) and, if given, out_offsets are
+ * written.  Host threads, no device work.  Errors: SW_EINVAL (index out of range,
+ * bad offsets, NULL), SW_ENOMEM.
+ */
+int32_t sw_subset_host(const uint8_t* codes, const int64_t* offsets, int64_t n_seqs, const int64_t* ids,
+                       int64_t n_ids, uint8_t* out_codes, int64_t* out_offsets, int64_t* n_out);
+
 #ifdef __cplusplus
 }
 #endif

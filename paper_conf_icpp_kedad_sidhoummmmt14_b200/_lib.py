@@ -17,7 +17,7 @@ SW_FLAG_TIMING = 1
 EXPORTS = ["sw_init", "sw_load_db", "sw_search", "sw_free_db", "sw_free", "sw_last_error",
            "sw_db_info", "sw_last_stats", "sw_set_option", "sw_encode_ascii", "sw_schedule_dual", "sw_align",
            "sw_encode_nucleotide", "sw_search_cpu", "sw_schedule_dual_dp", "sw_load_db_mapped",
-           "sw_assembly_create", "sw_assemble", "sw_assembly_free"]
+           "sw_assembly_create", "sw_assemble", "sw_assembly_free", "sw_subset_host"]
 
 
 class SWError(RuntimeError):
@@ -93,6 +93,8 @@ def lib() -> ctypes.CDLL:
     L.sw_assembly_create.argtypes = [V, V, I32, V, I64, V, I64, I32, I64, P(V)]
     L.sw_assemble.restype = I32
     L.sw_assemble.argtypes = [V, V, I64, V, V]
+    L.sw_subset_host.restype = I32
+    L.sw_subset_host.argtypes = [V, V, I64, V, I64, V, V, P(I64)]
     L.sw_assembly_free.restype = I32
     L.sw_assembly_free.argtypes = [V]
     _lib = L

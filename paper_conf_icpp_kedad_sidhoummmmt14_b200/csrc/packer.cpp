@@ -11,6 +11,7 @@
 //     (low byte = id0's residue, high byte = id1's), padded to a multiple of 4
 //     columns with PAD = alphabet_size, 4 columns = one 8-byte load;
 //   * pairs [0, n_long) are longer than t_long (launched separately).
+#include <cstring>
 #include <algorithm>
 #include <atomic>
 #include <stdexcept>
@@ -24,6 +25,7 @@
 namespace swdual {
 
 static unsigned n_threads() { return std::max(1u, std::min(16u, std::thread::hardware_concurrency())); }
+unsigned n_threads_host() { return n_threads(); }
 
 void pack_db(const uint8_t* codes, const int64_t* offsets, int64_t n_seqs, int alpha, int64_t t_long, Packed& P,
              bool nib) {
@@ -149,6 +151,42 @@ extern "C" int32_t sw_pack_db_host(const uint8_t* codes, const int64_t* offsets,
     return SW_OK;
   } catch (const std::invalid_argument&) {
     return SW_EINVAL;
+  } catch (...) {
+    return SW_ENOMEM;
+  }
+}
+
+// Host-only gather of selected sequences (the shard cut of the multi-GPU layer):
+// out_codes / out_offsets receive sequences ids[0..n_ids) in that order.  Two-phase:
+// out_codes == NULL returns the residue count in *n_out (offsets are filled when
+// out_offsets != NULL).  Copies run on the host's threads (C5 shards: billions of
+// residues, where an index-array gather would need 8 bytes per residue).
+extern "C" int32_t sw_subset_host(const uint8_t* codes, const int64_t* offsets, int64_t n_seqs, const int64_t* ids,
+                                  int64_t n_ids, uint8_t* out_codes, int64_t* out_offsets, int64_t* n_out) {
+  try {
+    if (n_ids < 0 || n_seqs < 0 || (n_ids > 0 && !ids) || (n_seqs > 0 && !offsets)) return SW_EINVAL;
+    std::vector<int64_t> off(size_t(n_ids) + 1, 0);
+    for (int64_t k = 0; k < n_ids; ++k) {
+      const int64_t d = ids[k];
+      if (d < 0 || d >= n_seqs) return SW_EINVAL;
+      const int64_t L = offsets[d + 1] - offsets[d];
+      if (L < 0) return SW_EINVAL;
+      off[size_t(k) + 1] = off[size_t(k)] + L;
+    }
+    if (n_out) *n_out = off.back();
+    if (out_offsets) std::copy(off.begin(), off.end(), out_offsets);
+    if (!out_codes) return SW_OK;
+    if (off.back() > 0 && !codes) return SW_EINVAL;
+    const unsigned nt = swdual::n_threads_host();
+    std::vector<std::thread> th;
+    for (unsigned t = 0; t < nt; ++t)
+      th.emplace_back([&, t] {
+        const int64_t a = n_ids * t / nt, b = n_ids * (t + 1) / nt;
+        for (int64_t k = a; k < b; ++k)
+          std::memcpy(out_codes + off[size_t(k)], codes + offsets[ids[k]], size_t(off[size_t(k) + 1] - off[size_t(k)]));
+      });
+    for (auto& x : th) x.join();
+    return SW_OK;
   } catch (...) {
     return SW_ENOMEM;
   }

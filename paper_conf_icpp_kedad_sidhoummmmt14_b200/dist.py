@@ -40,19 +40,23 @@ def shard_cut(offsets, n_shards: int) -> list[np.ndarray]:
 
 
 def subset(codes, offsets, idx):
-    """(codes, offsets) of the sequences idx, in that order."""
-    off = np.asarray(offsets, dtype=np.int64)
-    idx = np.asarray(idx, dtype=np.int64)
-    lens = off[idx + 1] - off[idx]
+    """(codes, offsets) of the sequences idx, in that order (sw_subset_host: a
+    threaded host gather, no per-residue index array)."""
+    import ctypes
+    from ._lib import check, lib
+    off = np.ascontiguousarray(offsets, dtype=np.int64)
+    idx = np.ascontiguousarray(idx, dtype=np.int64)
+    codes = np.ascontiguousarray(codes, dtype=np.uint8)
     new_off = np.zeros(len(idx) + 1, dtype=np.int64)
-    np.cumsum(lens, out=new_off[1:])
-    if len(idx) == 0:
-        return np.zeros(0, np.uint8), new_off
-    starts = off[idx]
-    # gather residues
-    rep = np.repeat(starts - new_off[:-1], lens)
-    src = np.arange(int(new_off[-1]), dtype=np.int64) + rep
-    return np.asarray(codes)[src], new_off
+    n = ctypes.c_int64()
+    vp = lambda a: a.ctypes.data_as(ctypes.c_void_p) if a.size else None  # noqa: E731
+    check(lib().sw_subset_host(vp(codes), vp(off), len(off) - 1, vp(idx), len(idx), None, vp(new_off),
+                               ctypes.byref(n)))
+    out = np.empty(int(n.value), dtype=np.uint8)
+    if len(idx):
+        check(lib().sw_subset_host(vp(codes), vp(off), len(off) - 1, vp(idx), len(idx), vp(out), vp(new_off),
+                                   ctypes.byref(n)))
+    return out, new_off
 
 
 @dataclass

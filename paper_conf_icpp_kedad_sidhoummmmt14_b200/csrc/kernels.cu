@@ -156,11 +156,17 @@ struct SubLanes {
 // (written in one pass, read in the next).  Long items: a shared-memory ring
 // between two concurrently running warps (producer progress / consumer progress
 // counters, LONG_RING steps of slack) or, for the round wrap, a global row.
-// Every ring, and its producer-progress counter, lives in the CONSUMER's CTA; the
-// consumer-progress counter lives in the PRODUCER's CTA.  Each warp therefore
-// polls only its own CTA's shared memory, and writes -- ring cells, progress,
-// consumption -- go through generic pointers that may name another CTA of the
-// thread-block cluster (distributed shared memory), with cluster-scope ordering.
+// Every ring lives in the CONSUMER's CTA and the consumer-progress counter in the
+// PRODUCER's CTA, so each warp polls only its own CTA's shared memory; writes --
+// ring cells, consumption -- go through generic pointers that may name another
+// CTA of the thread-block cluster (distributed shared memory).  A ring cell is one
+// 8-byte store (single-copy atomic) of (H, F) whose bit 15 of both H halves
+// carries the parity of its lap (step index / LONG_RING): the consumer spins on
+// the cell itself until the parity matches, so no progress counter, fence or L1
+// invalidation sits on the ring path (H <= 32767 leaves bit 15 free; a wrapped
+// int16 value only occurs in a pair already flagged for the int32 re-score).
+// The round wrap goes through a global row plus a progress counter (release
+// store, relaxed poll, L2 reads).
 struct Chain {
   bool in_ring, out_ring;    // rings (shared memory) or global rows
   uint32_t in_sring;         // this CTA's shared-window address of the input ring
@@ -172,11 +178,12 @@ struct Chain {
   int in_base, out_base;     // step index (monotone across rounds) of the producer's / this warp's step 0
   const uint2* grow_in;      // global input row (round wrap)
   uint2* grow_out;           // global output row (round wrap)
+  bool cluster;              // the wrap counter may be in another CTA (cluster-scope release)
 };
 
-__device__ __forceinline__ int ld_acquire_cluster(const int* p) {
+__device__ __forceinline__ int ld_relaxed_cluster(const int* p) {
   int v;
-  asm volatile("ld.acquire.cluster.b32 %0, [%1];" : "=r"(v) : "l"(p) : "memory");
+  asm volatile("ld.relaxed.cluster.b32 %0, [%1];" : "=r"(v) : "l"(p) : "memory");
   return v;
 }
 __device__ __forceinline__ void st_release_cluster(int* p, int v) {
@@ -214,13 +221,14 @@ __device__ __forceinline__ void sts64(uint32_t a, uint2 v) {
   asm volatile("st.shared.v2.u32 [%0], {%1, %2};" :: "r"(a), "r"(v.x), "r"(v.y) : "memory");
 }
 
-// Warp-uniform spin until *p >= need: lane `who` (the lane whose later shared
-// memory accesses the counter orders) polls with acquire, the value is broadcast.
+// Warp-uniform spin until *p >= need: lane `who` polls (relaxed: the counters
+// only gate WAR reuse of ring cells and the wrap row read through L2, see Chain),
+// the value is broadcast.
 __device__ __forceinline__ void wait_geq(const int* p, int need, int& seen, int who) {
   if (seen >= need) return;
   for (;;) {
     int v = 0;
-    if ((threadIdx.x & 31) == who) v = ld_acquire_cluster(p);
+    if ((threadIdx.x & 31) == who) v = ld_relaxed_cluster(p);
     v = __shfl_sync(FULL, v, who);
     if (v >= need) { seen = v; return; }
     __nanosleep(32);
@@ -271,12 +279,21 @@ __device__ __forceinline__ void strip_pass(const uint8_t* sprof, int LS, int LB,
     if (rd) {
       if constexpr (LINKED) {
         if (ch.in_ring) {
+          // the cell of producer step x, once written (lap parity in bit 15 of H); steps
+          // past the producer's last one feed PAD columns only: zero
+          auto cell = [&](int x) -> uint2 {
+            if (x >= ch.in_base + T) return z2;
+            const uint32_t a = ch.in_sring + uint32_t((x & (LONG_RING - 1)) * 8);
+            const uint32_t want = ((x / LONG_RING) & 1) ? 0x80008000u : 0u;
+            uint2 v = lds64(a);
+            while ((v.x & 0x80008000u) != want) {
+              __nanosleep(20);
+              v = lds64(a);
+            }
+            return make_uint2(v.x & 0x7fff7fffu, v.y);
+          };
           const int x = ch.in_base + t0 + ioff;  // 3 mod 4 (ioff = 63): the 4 cells one by one
-          const uint32_t a0 = ch.in_sring + uint32_t((x & (LONG_RING - 1)) * 8);
-          const uint32_t a1 = ch.in_sring + uint32_t(((x + 1) & (LONG_RING - 1)) * 8);
-          const uint32_t a2 = ch.in_sring + uint32_t(((x + 2) & (LONG_RING - 1)) * 8);
-          const uint32_t a3 = ch.in_sring + uint32_t(((x + 3) & (LONG_RING - 1)) * 8);
-          b0 = lds64(a0); b1 = lds64(a1); b2 = lds64(a2); b3 = lds64(a3);
+          b0 = cell(x); b1 = cell(x + 1); b2 = cell(x + 2); b3 = cell(x + 3);
         } else {
           const uint2* g = ch.grow_in + t0 + ioff;
           b0 = __ldcg(g); b1 = __ldcg(g + 1); b2 = __ldcg(g + 2); b3 = __ldcg(g + 3);
@@ -291,7 +308,7 @@ __device__ __forceinline__ void strip_pass(const uint8_t* sprof, int LS, int LB,
   // long items: progress this warp's consumer needs before block t0's prefetch
   auto wait_in = [&](int t0) {
     if constexpr (LINKED) {
-      if (rd) wait_geq(ch.in_prog, ch.in_base + min(t0 + 4 + ioff + LINK_LAG, L + VG), seen_in, 0);
+      if (rd && !ch.in_ring) wait_geq(ch.in_prog, ch.in_base + min(t0 + 4 + ioff + LINK_LAG, L + VG), seen_in, 0);
     }
   };
   uint2 cw = make_uint2(pad4, pad4);
@@ -368,7 +385,11 @@ __device__ __forceinline__ void strip_pass(const uint8_t* sprof, int LS, int LB,
       }
       if (wr && tail) {
         if constexpr (LINKED) {
-          if (ch.out_ring) st_generic_v2(ch.out_ring_ptr + ((ch.out_base + t0 + j) & (LONG_RING - 1)), make_uint2(sH, sF));
+          if (ch.out_ring) {
+            const int g = ch.out_base + t0 + j;
+            const uint32_t tag = ((g / LONG_RING) & 1) ? 0x80008000u : 0u;
+            st_generic_v2(ch.out_ring_ptr + (g & (LONG_RING - 1)), make_uint2((sH & 0x7fff7fffu) | tag, sF));
+          }
           else __stcg(ch.grow_out + t0 + j, make_uint2(sH, sF));
         } else {
           wp[t0 + j] = make_uint2(sH, sF);
@@ -377,8 +398,10 @@ __device__ __forceinline__ void strip_pass(const uint8_t* sprof, int LS, int LB,
     }
     if constexpr (LINKED) {
       // progress, every 8 columns: release orders this lane's ring writes before the counter
-      if (wr && tail && ((((t0 >> 2) + 1) % (SW_PROG_EVERY / 4)) == 0 || t0 + 4 >= T))
-        st_release_cluster(ch.out_prog, ch.out_base + t0 + 4);
+      if (wr && tail && !ch.out_ring && ((((t0 >> 2) + 1) % (SW_PROG_EVERY / 4)) == 0 || t0 + 4 >= T)) {
+        if (ch.cluster) st_release_cluster(ch.out_prog, ch.out_base + t0 + 4);
+        else st_release_cta(ch.out_prog, ch.out_base + t0 + 4);
+      }
       // consumption: block t0's ring cells were used above (their loads completed), so a
       // relaxed store suffices -- the producer only overwrites cells below this index
       if (rd && ch.in_ring && lead && (((t0 >> 2) & 1) || t0 + 4 >= T))
@@ -576,6 +599,8 @@ __device__ __forceinline__ void long_item(const LongArgs& a, int item, uint8_t* 
   uint2* wrap = a.wrap + (size_t)(blockIdx.x / KC) * a.wcap;
   if (tid < W) { sh.prog[tid] = -1; sh.cons[tid] = 0; }
   if (tid == 0) sh.wprog = -1;
+  for (int i = tid; i < W * LONG_RING; i += blockDim.x)  // every cell "written in lap -1"
+    rings[i] = make_uint2(0x80008000u, 0u);
   if (crank == 0)
     for (int i = tid; i < 2 * W * 4; i += blockDim.x) sh.pbest[i] = 0;
   csync();  // every CTA reset before any remote write of this item
@@ -611,11 +636,11 @@ __device__ __forceinline__ void long_item(const LongArgs& a, int item, uint8_t* 
     __syncwarp();
     const bool rd = s > 0, wr = s + 1 < ns;
     Chain ch{};
+    ch.cluster = KC > 1;
     ch.out_base = r * T;
     ch.in_ring = j > 0;
     if (j > 0) {  // input: ring of the producer warp (same round), held here
       ch.in_sring = static_cast<uint32_t>(__cvta_generic_to_shared(rings + (size_t)warp * LONG_RING));
-      ch.in_prog = &sh.prog[warp];
       ch.in_cons = map_rank(&sh.cons[gprod % W], uint32_t(gprod / W));
       ch.in_base = r * T;
     } else {      // input: the wrap row of the previous round
@@ -626,7 +651,6 @@ __device__ __forceinline__ void long_item(const LongArgs& a, int item, uint8_t* 
     ch.out_ring = j < GS - 1;
     if (j < GS - 1) {
       ch.out_ring_ptr = map_rank(rings + (size_t)(gcons % W) * LONG_RING, uint32_t(gcons / W));
-      ch.out_prog = map_rank(&sh.prog[gcons % W], uint32_t(gcons / W));
       ch.out_cons = &sh.cons[warp];
     } else {      // only reached when ns > TW (P = 1): the round wrap
       ch.grow_out = wrap;

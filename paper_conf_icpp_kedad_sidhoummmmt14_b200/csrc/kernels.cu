@@ -284,7 +284,7 @@ __device__ __forceinline__ void strip_pass(const uint8_t* sprof, int LS, int LB,
           auto cell = [&](int x) -> uint2 {
             if (x >= ch.in_base + T) return z2;
             const uint32_t a = ch.in_sring + uint32_t((x & (LONG_RING - 1)) * 8);
-            const uint32_t want = ((x / LONG_RING) & 1) ? 0x80008000u : 0u;
+            const uint32_t want = ((uint32_t(x) / LONG_RING) & 1u) ? 0x80008000u : 0u;
             uint2 v = lds64(a);
             while ((v.x & 0x80008000u) != want) {
               __nanosleep(20);
@@ -313,6 +313,16 @@ __device__ __forceinline__ void strip_pass(const uint8_t* sprof, int LS, int LB,
   };
   uint2 cw = make_uint2(pad4, pad4);
   uint2 tb0 = z2, tb1 = z2, tb2 = z2, tb3 = z2;
+  if constexpr (LINKED) {
+    // ring input: start once the producer is LINK_LAG steps past our first block, so the
+    // two warps run decoupled (later cells are then rarely waited for)
+    if (rd && ch.in_ring && lead && L > 0) {
+      const int x = ch.in_base + min(ioff + 7 + LINK_LAG, T - 1);
+      const uint32_t a = ch.in_sring + uint32_t((x & (LONG_RING - 1)) * 8);
+      const uint32_t want = ((uint32_t(x) / LONG_RING) & 1u) ? 0x80008000u : 0u;
+      while ((lds64(a).x & 0x80008000u) != want) __nanosleep(32);
+    }
+  }
   if (L > 0) {
     wait_in(0);
     if (lead) load_block(0, cw, tb0, tb1, tb2, tb3);
@@ -387,7 +397,7 @@ __device__ __forceinline__ void strip_pass(const uint8_t* sprof, int LS, int LB,
         if constexpr (LINKED) {
           if (ch.out_ring) {
             const int g = ch.out_base + t0 + j;
-            const uint32_t tag = ((g / LONG_RING) & 1) ? 0x80008000u : 0u;
+            const uint32_t tag = ((uint32_t(g) / LONG_RING) & 1u) ? 0x80008000u : 0u;
             st_generic_v2(ch.out_ring_ptr + (g & (LONG_RING - 1)), make_uint2((sH & 0x7fff7fffu) | tag, sF));
           }
           else __stcg(ch.grow_out + t0 + j, make_uint2(sH, sF));
@@ -757,6 +767,8 @@ __global__ void __launch_bounds__(LONG_W * 32, 2) long_kernel(LongArgs al) {
     if (crank == 0 && threadIdx.x == 0) sh.item = atomicAdd(al.work_counter, 1);
     if (KC > 1) cluster_sync_all(); else __syncthreads();
     const int item = *map_rank(&sh.item, 0u);
+    // every CTA has read the item before CTA 0 may exit (its shared memory would vanish)
+    if (KC > 1) cluster_sync_all(); else __syncthreads();
     if (item >= al.n_items) break;
     long_item<NIB>(al, item, smem, sh);  // ends with a cluster barrier: sh.item may be rewritten
   }

@@ -281,19 +281,12 @@ __device__ __forceinline__ void strip_pass(const uint8_t* sprof, int LS, int LB,
         if (ch.in_ring) {
           // the cell of producer step x, once written (lap parity in bit 15 of H); steps
           // past the producer's last one feed PAD columns only: zero
-          auto cell = [&](int x) -> uint2 {
-            if (x >= ch.in_base + T) return z2;
-            const uint32_t a = ch.in_sring + uint32_t((x & (LONG_RING - 1)) * 8);
-            const uint32_t want = ((uint32_t(x) / LONG_RING) & 1u) ? 0x80008000u : 0u;
-            uint2 v = lds64(a);
-            while ((v.x & 0x80008000u) != want) {
-              __nanosleep(20);
-              v = lds64(a);
-            }
-            return make_uint2(v.x & 0x7fff7fffu, v.y);
-          };
+          // (prefetched without a check: the tags are verified when the block is used)
           const int x = ch.in_base + t0 + ioff;  // 3 mod 4 (ioff = 63): the 4 cells one by one
-          b0 = cell(x); b1 = cell(x + 1); b2 = cell(x + 2); b3 = cell(x + 3);
+          b0 = lds64(ch.in_sring + uint32_t((x & (LONG_RING - 1)) * 8));
+          b1 = lds64(ch.in_sring + uint32_t(((x + 1) & (LONG_RING - 1)) * 8));
+          b2 = lds64(ch.in_sring + uint32_t(((x + 2) & (LONG_RING - 1)) * 8));
+          b3 = lds64(ch.in_sring + uint32_t(((x + 3) & (LONG_RING - 1)) * 8));
         } else {
           const uint2* g = ch.grow_in + t0 + ioff;
           b0 = __ldcg(g); b1 = __ldcg(g + 1); b2 = __ldcg(g + 2); b3 = __ldcg(g + 3);
@@ -330,6 +323,24 @@ __device__ __forceinline__ void strip_pass(const uint8_t* sprof, int LS, int LB,
   __syncwarp();
   for (int t0 = 0; t0 < T; t0 += 4) {
     const uint2 cwc = cw;
+    if constexpr (LINKED) {
+      // ring input: every prefetched cell must carry its lap's parity; a cell read before
+      // the producer wrote it is read again (rare: the consumer runs LINK_LAG behind);
+      // cells past the producer's last step feed PAD columns only and are zeroed
+      if (rd && ch.in_ring && lead && t0 < L) {
+        const int x = ch.in_base + t0 + ioff;
+        auto fix = [&](uint2& v, int xi) {
+          if (xi >= ch.in_base + T) { v = z2; return; }
+          const uint32_t want = ((uint32_t(xi) / LONG_RING) & 1u) ? 0x80008000u : 0u;
+          if ((v.x & 0x80008000u) != want) {
+            const uint32_t a = ch.in_sring + uint32_t((xi & (LONG_RING - 1)) * 8);
+            do { __nanosleep(20); v = lds64(a); } while ((v.x & 0x80008000u) != want);
+          }
+          v.x &= 0x7fff7fffu;
+        };
+        fix(tb0, x); fix(tb1, x + 1); fix(tb2, x + 2); fix(tb3, x + 3);
+      }
+    }
     const uint2 c0 = tb0, c1 = tb1, c2 = tb2, c3 = tb3;
     if (t0 + 4 < L) wait_in(t0 + 4);
     if constexpr (LINKED) {

@@ -19,7 +19,7 @@ from __future__ import annotations
 import ctypes
 import os
 import subprocess
-import multiprocessing as mp
+from concurrent.futures import ThreadPoolExecutor
 
 import numpy as np
 
@@ -100,7 +100,9 @@ def gotoh_search(qcodes, qoff, dcodes, doff, S, gs: int, ge: int, procs: int = 1
     """scores[q][d] for every query x database pair (L196-201).
 
     procs > 1 splits the database into disjoint subsets scored by independent
-    single-threaded worker processes (each runs the same plain C loop).
+    worker threads (each runs the same plain, single-threaded C loop; ctypes
+    releases the GIL for the call).  Threads, not forked processes: forking a
+    process that already runs CUDA / torch threads can deadlock the child.
     """
     qcodes = np.ascontiguousarray(qcodes, dtype=np.uint8)
     dcodes = np.ascontiguousarray(dcodes, dtype=np.uint8)
@@ -121,9 +123,8 @@ def gotoh_search(qcodes, qoff, dcodes, doff, S, gs: int, ge: int, procs: int = 1
     jobs = [(qcodes, qoff, dcodes, doff, a, b, S, gs, ge) for a, b in zip(cuts[:-1], cuts[1:]) if b > a]
     out = np.zeros((nq, nd), dtype=np.int32)
     build()
-    ctx = mp.get_context("fork")
-    with ctx.Pool(procs) as pool:
-        for b0, b1, blk in pool.imap_unordered(_search_chunk, jobs):
+    with ThreadPoolExecutor(max_workers=procs) as pool:
+        for b0, b1, blk in pool.map(_search_chunk, jobs):
             out[:, b0:b1] = blk
     return out
 

@@ -122,7 +122,6 @@ struct sw_handle_s {
   int64_t opt_const_gaps = 1;   // gaps 10/2: the constant-gap kernel instantiations
   int64_t opt_nibble = 1;       // alphabets <= 15: 4-bit DB stream
   int64_t opt_small_ctas = 1;   // latency-bound single-query searches: 32-thread CTAs
-  int64_t opt_long_cluster = 1; // long-only searches: thread-block clusters per long item
   int64_t opt_crit_min = CRIT_MIN_STEPS;                    // long-pair rule (see launch_all)
   int64_t opt_crit_pct = int64_t(CRIT_FRACTION * 100 + 0.5);
   int64_t opt_align_ws_mb = 2048;  // sw_align: traceback-code workspace per batch
@@ -372,8 +371,6 @@ int32_t sw_set_option(sw_handle_t h, const char* key, int64_t value) {
   } else if (k == "crit_pct") {
     if (value < 1) return set_err(h, SW_EINVAL, "crit_pct must be >= 1");
     h->opt_crit_pct = value;
-  } else if (k == "long_cluster") {
-    h->opt_long_cluster = value;
   } else if (k == "small_ctas") {
     h->opt_small_ctas = value;
   } else if (k == "nibble") {
@@ -718,17 +715,6 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
     if (sl.nlong > 0) any_long = true;
   }
   const bool combined = any_long && any_m0 && !any_q2;
-  // Long-only searches (C4-like): the long kernel runs alone; very tall queries split
-  // each pair over a thread-block cluster of KC CTAs (co-scheduled, so the chained
-  // warps of different CTAs may wait on each other across rounds), the smallest KC
-  // with at most 3 rounds for the tallest query -- the longest item's critical path.
-  int KC = 1;
-  if (any_long && !any_q2 && !any_m0 && h->opt_long_cluster != 0) {
-    int ns_max = 1;
-    for (size_t k = 0; k < order.size(); ++k)
-      if (qnlong[k] > 0) ns_max = std::max(ns_max, gl[k].n_strips);
-    while (KC < 4 && (ns_max + KC * W - 1) / (KC * W) > 3) ++KC;
-  }
   if (small_ctas && !combined) {  // (a combined launch needs whole CTAs for its long items)
     NT0 = 32;
     NG0 = NT0 / G0;
@@ -750,10 +736,9 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
     d.n_strips = gl[k].n_strips;
     d.qidx = order[k];
     d.n_long = nl;
-    const int TW = KC * W;  // warps per long item
-    d.pack = (combined || gl[k].n_strips >= TW) ? 1 : TW / gl[k].n_strips;
+    d.pack = (combined || gl[k].n_strips >= W) ? 1 : W / gl[k].n_strips;
     // item cost: rounds x the item's longest pair (pairs are sorted longest first)
-    const int GS = gl[k].n_strips >= TW ? TW : gl[k].n_strips;
+    const int GS = gl[k].n_strips >= W ? W : gl[k].n_strips;
     const double rounds = double((gl[k].n_strips + GS - 1) / GS);
     for (int it = 0; it * d.pack < nl; ++it)
       litems.push_back({rounds * double(db->pairs[size_t(it * d.pack)].len + 64), int(ldesc.size()), it});
@@ -907,7 +892,7 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
     al.n_items = int(long_items);
     al.lmap = h->lmap.as<int2>();
     al.SBL = l0.SB; al.LSL = l0.LS; al.LBL = l0.LB;
-    smem_long = W * LONG_RING * int(sizeof(uint2)) + W * l0.SB;
+    smem_long = (W - 1) * LONG_RING * int(sizeof(uint2)) + W * l0.SB;
     al.wcap = max_long + 64 + 8;
     al.stream = db->stream.as<uint16_t>();
     al.pairs = db->dpairs.as<PairRec>();
@@ -923,10 +908,9 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
   if (long_items > 0 && !combined) {
     int smem = smem_long;
     if (fork) smem = std::max(smem, 200 * 1024);  // SM-exclusive (see above)
-    const int ncl = long_max_clusters(smem, nib, KC);
-    if (ncl <= 0) fail(SW_ECUDA, "long-pair kernel does not fit on an SM");
-    const int64_t slots = KC > 1 ? int64_t(ncl) : int64_t(ncl) * h->sms;  // resident clusters (or CTAs)
-    const int grid = int(std::max<int64_t>(1, std::min<int64_t>(long_items, slots))) * KC;
+    const int occ = long_max_ctas_per_sm(smem, nib);
+    if (occ <= 0) fail(SW_ECUDA, "long-pair kernel does not fit on an SM");
+    const int grid = int(std::max<int64_t>(1, std::min<int64_t>(long_items, int64_t(occ) * h->sms)));
     SW_CK(h->wrap.ensure(size_t(grid) * al.wcap * sizeof(uint2)));
     al.wrap = h->wrap.as<uint2>();
     cudaStream_t lst = c.st;
@@ -944,7 +928,7 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
     }
     std::pair<cudaEvent_t, cudaEvent_t>* ev = nullptr;
     record_begin(h, c.timing, 1, lst, ev);
-    SW_CK(launch_long(grid, smem, al, lst, nib, KC));
+    SW_CK(launch_long(grid, smem, al, lst, nib));
     if (ev) SW_CK(cudaEventRecord(ev->second, lst));
     if (fork) SW_CK(cudaEventRecord(h->ev_join, lst));
     ++out.launches;

@@ -32,13 +32,7 @@ constexpr int8_t PAD_SCORE = -64;  // S[.][PAD] = S[PAD][.] <= 0 (reading R-12)
 // Intra-task mode: a strip starts consuming the row above only once its
 // producer is this many columns ahead, so producer and consumer warps of a
 // chain run decoupled instead of in lock-step (the consumer then rarely waits).
-#ifndef SW_LINK_LAG
-#define SW_LINK_LAG 32
-#endif
-#ifndef SW_PROG_EVERY
-#define SW_PROG_EVERY 8   // columns between producer-progress releases of the long links
-#endif
-constexpr int LINK_LAG = SW_LINK_LAG;
+constexpr int LINK_LAG = 32;
 constexpr int RESCORE_LAG = 16;  // re-score chains: one round per CTA, short lag keeps the critical path short
 
 // ---------------------------------------------------------------------------
@@ -156,79 +150,30 @@ struct SubLanes {
 // (written in one pass, read in the next).  Long items: a shared-memory ring
 // between two concurrently running warps (producer progress / consumer progress
 // counters, LONG_RING steps of slack) or, for the round wrap, a global row.
-// Every ring lives in the CONSUMER's CTA and the consumer-progress counter in the
-// PRODUCER's CTA, so each warp polls only its own CTA's shared memory; writes --
-// ring cells, consumption -- go through generic pointers that may name another
-// CTA of the thread-block cluster (distributed shared memory).  A ring cell is one
-// 8-byte store (single-copy atomic) of (H, F) whose bit 15 of both H halves
-// carries the parity of its lap (step index / LONG_RING): the consumer spins on
-// the cell itself until the parity matches, so no progress counter, fence or L1
-// invalidation sits on the ring path (H <= 32767 leaves bit 15 free; a wrapped
-// int16 value only occurs in a pair already flagged for the int32 re-score).
-// The round wrap goes through a global row plus a progress counter (release
-// store, relaxed poll, L2 reads).
 struct Chain {
   bool in_ring, out_ring;    // rings (shared memory) or global rows
-  uint32_t in_sring;         // this CTA's shared-window address of the input ring
-  uint2* out_ring_ptr;       // the consumer's ring (generic; DSMEM when in another CTA)
-  const int* in_prog;        // producer progress (steps written, monotone across rounds), local
-  int* in_cons;              // this warp's consumption of its input, in the producer's CTA (generic)
-  int* out_prog;             // this warp's output progress, in the consumer's CTA (generic)
-  const int* out_cons;       // consumption of this warp's output by its consumer, local
+  uint32_t in_sring, out_sring;  // shared-window addresses of the rings
+  int* in_prog;              // producer progress (steps written, monotone across rounds), shared
+  int* in_cons;              // this warp's consumption of its input, published for the producer
+  int* out_prog;             // this warp's output progress
+  const int* out_cons;       // consumption of this warp's output by its consumer
   int in_base, out_base;     // step index (monotone across rounds) of the producer's / this warp's step 0
   const uint2* grow_in;      // global input row (round wrap)
   uint2* grow_out;           // global output row (round wrap)
-  bool cluster;              // the wrap counter may be in another CTA (cluster-scope release)
 };
-
-__device__ __forceinline__ int ld_relaxed_cluster(const int* p) {
-  int v;
-  asm volatile("ld.relaxed.cluster.b32 %0, [%1];" : "=r"(v) : "l"(p) : "memory");
-  return v;
-}
-__device__ __forceinline__ void st_release_cluster(int* p, int v) {
-  asm volatile("st.release.cluster.b32 [%0], %1;" :: "l"(p), "r"(v) : "memory");
-}
-__device__ __forceinline__ void st_relaxed_cluster(int* p, int v) {
-  asm volatile("st.relaxed.cluster.b32 [%0], %1;" :: "l"(p), "r"(v) : "memory");
-}
-__device__ __forceinline__ void st_generic_v2(uint2* p, uint2 v) {
-  asm volatile("st.v2.u32 [%0], {%1, %2};" :: "l"(p), "r"(v.x), "r"(v.y) : "memory");
-}
-__device__ __forceinline__ uint32_t cluster_ctarank() {
-  uint32_t r;
-  asm volatile("mov.u32 %0, %%cluster_ctarank;" : "=r"(r));
-  return r;
-}
-__device__ __forceinline__ uint32_t cluster_nctarank() {
-  uint32_t r;
-  asm volatile("mov.u32 %0, %%cluster_nctarank;" : "=r"(r));
-  return r;
-}
-// generic address of `p` (this CTA's shared memory) in CTA `rank` of the cluster
-template <class T>
-__device__ __forceinline__ T* map_rank(T* p, uint32_t rank) {
-  uint64_t out;
-  asm volatile("mapa.u64 %0, %1, %2;" : "=l"(out) : "l"(reinterpret_cast<uint64_t>(p)), "r"(rank));
-  return reinterpret_cast<T*>(out);
-}
-__device__ __forceinline__ void cluster_sync_all() {
-  asm volatile("barrier.cluster.arrive.release.aligned;\nbarrier.cluster.wait.acquire.aligned;" ::: "memory");
-}
 
 __device__ __forceinline__ uint4 lds128v(uint32_t a) { return lds128(a); }
 __device__ __forceinline__ void sts64(uint32_t a, uint2 v) {
   asm volatile("st.shared.v2.u32 [%0], {%1, %2};" :: "r"(a), "r"(v.x), "r"(v.y) : "memory");
 }
 
-// Warp-uniform spin until *p >= need: lane `who` polls (relaxed: the counters
-// only gate WAR reuse of ring cells and the wrap row read through L2, see Chain),
-// the value is broadcast.
+// Warp-uniform spin until *p >= need: lane `who` (the lane whose later shared
+// memory accesses the counter orders) polls with acquire, the value is broadcast.
 __device__ __forceinline__ void wait_geq(const int* p, int need, int& seen, int who) {
   if (seen >= need) return;
   for (;;) {
     int v = 0;
-    if ((threadIdx.x & 31) == who) v = ld_relaxed_cluster(p);
+    if ((threadIdx.x & 31) == who) v = ld_acquire_cta(p);
     v = __shfl_sync(FULL, v, who);
     if (v >= need) { seen = v; return; }
     __nanosleep(32);
@@ -279,14 +224,12 @@ __device__ __forceinline__ void strip_pass(const uint8_t* sprof, int LS, int LB,
     if (rd) {
       if constexpr (LINKED) {
         if (ch.in_ring) {
-          // the cell of producer step x, once written (lap parity in bit 15 of H); steps
-          // past the producer's last one feed PAD columns only: zero
-          // (prefetched without a check: the tags are verified when the block is used)
           const int x = ch.in_base + t0 + ioff;  // 3 mod 4 (ioff = 63): the 4 cells one by one
-          b0 = lds64(ch.in_sring + uint32_t((x & (LONG_RING - 1)) * 8));
-          b1 = lds64(ch.in_sring + uint32_t(((x + 1) & (LONG_RING - 1)) * 8));
-          b2 = lds64(ch.in_sring + uint32_t(((x + 2) & (LONG_RING - 1)) * 8));
-          b3 = lds64(ch.in_sring + uint32_t(((x + 3) & (LONG_RING - 1)) * 8));
+          const uint32_t a0 = ch.in_sring + uint32_t((x & (LONG_RING - 1)) * 8);
+          const uint32_t a1 = ch.in_sring + uint32_t(((x + 1) & (LONG_RING - 1)) * 8);
+          const uint32_t a2 = ch.in_sring + uint32_t(((x + 2) & (LONG_RING - 1)) * 8);
+          const uint32_t a3 = ch.in_sring + uint32_t(((x + 3) & (LONG_RING - 1)) * 8);
+          b0 = lds64(a0); b1 = lds64(a1); b2 = lds64(a2); b3 = lds64(a3);
         } else {
           const uint2* g = ch.grow_in + t0 + ioff;
           b0 = __ldcg(g); b1 = __ldcg(g + 1); b2 = __ldcg(g + 2); b3 = __ldcg(g + 3);
@@ -301,21 +244,11 @@ __device__ __forceinline__ void strip_pass(const uint8_t* sprof, int LS, int LB,
   // long items: progress this warp's consumer needs before block t0's prefetch
   auto wait_in = [&](int t0) {
     if constexpr (LINKED) {
-      if (rd && !ch.in_ring) wait_geq(ch.in_prog, ch.in_base + min(t0 + 4 + ioff + LINK_LAG, L + VG), seen_in, 0);
+      if (rd) wait_geq(ch.in_prog, ch.in_base + min(t0 + 4 + ioff + LINK_LAG, L + VG), seen_in, 0);
     }
   };
   uint2 cw = make_uint2(pad4, pad4);
   uint2 tb0 = z2, tb1 = z2, tb2 = z2, tb3 = z2;
-  if constexpr (LINKED) {
-    // ring input: start once the producer is LINK_LAG steps past our first block, so the
-    // two warps run decoupled (later cells are then rarely waited for)
-    if (rd && ch.in_ring && lead && L > 0) {
-      const int x = ch.in_base + min(ioff + 7 + LINK_LAG, T - 1);
-      const uint32_t a = ch.in_sring + uint32_t((x & (LONG_RING - 1)) * 8);
-      const uint32_t want = ((uint32_t(x) / LONG_RING) & 1u) ? 0x80008000u : 0u;
-      while ((lds64(a).x & 0x80008000u) != want) __nanosleep(32);
-    }
-  }
   if (L > 0) {
     wait_in(0);
     if (lead) load_block(0, cw, tb0, tb1, tb2, tb3);
@@ -323,24 +256,6 @@ __device__ __forceinline__ void strip_pass(const uint8_t* sprof, int LS, int LB,
   __syncwarp();
   for (int t0 = 0; t0 < T; t0 += 4) {
     const uint2 cwc = cw;
-    if constexpr (LINKED) {
-      // ring input: every prefetched cell must carry its lap's parity; a cell read before
-      // the producer wrote it is read again (rare: the consumer runs LINK_LAG behind);
-      // cells past the producer's last step feed PAD columns only and are zeroed
-      if (rd && ch.in_ring && lead && t0 < L) {
-        const int x = ch.in_base + t0 + ioff;
-        auto fix = [&](uint2& v, int xi) {
-          if (xi >= ch.in_base + T) { v = z2; return; }
-          const uint32_t want = ((uint32_t(xi) / LONG_RING) & 1u) ? 0x80008000u : 0u;
-          if ((v.x & 0x80008000u) != want) {
-            const uint32_t a = ch.in_sring + uint32_t((xi & (LONG_RING - 1)) * 8);
-            do { __nanosleep(20); v = lds64(a); } while ((v.x & 0x80008000u) != want);
-          }
-          v.x &= 0x7fff7fffu;
-        };
-        fix(tb0, x); fix(tb1, x + 1); fix(tb2, x + 2); fix(tb3, x + 3);
-      }
-    }
     const uint2 c0 = tb0, c1 = tb1, c2 = tb2, c3 = tb3;
     if (t0 + 4 < L) wait_in(t0 + 4);
     if constexpr (LINKED) {
@@ -406,11 +321,7 @@ __device__ __forceinline__ void strip_pass(const uint8_t* sprof, int LS, int LB,
       }
       if (wr && tail) {
         if constexpr (LINKED) {
-          if (ch.out_ring) {
-            const int g = ch.out_base + t0 + j;
-            const uint32_t tag = ((uint32_t(g) / LONG_RING) & 1u) ? 0x80008000u : 0u;
-            st_generic_v2(ch.out_ring_ptr + (g & (LONG_RING - 1)), make_uint2((sH & 0x7fff7fffu) | tag, sF));
-          }
+          if (ch.out_ring) sts64(ch.out_sring + uint32_t(((ch.out_base + t0 + j) & (LONG_RING - 1)) * 8), make_uint2(sH, sF));
           else __stcg(ch.grow_out + t0 + j, make_uint2(sH, sF));
         } else {
           wp[t0 + j] = make_uint2(sH, sF);
@@ -419,18 +330,15 @@ __device__ __forceinline__ void strip_pass(const uint8_t* sprof, int LS, int LB,
     }
     if constexpr (LINKED) {
       // progress, every 8 columns: release orders this lane's ring writes before the counter
-      if (wr && tail && !ch.out_ring && ((((t0 >> 2) + 1) % (SW_PROG_EVERY / 4)) == 0 || t0 + 4 >= T)) {
-        if (ch.cluster) st_release_cluster(ch.out_prog, ch.out_base + t0 + 4);
-        else st_release_cta(ch.out_prog, ch.out_base + t0 + 4);
-      }
+      if (wr && tail && (((t0 >> 2) & 1) || t0 + 4 >= T)) st_release_cta(ch.out_prog, ch.out_base + t0 + 4);
       // consumption: block t0's ring cells were used above (their loads completed), so a
       // relaxed store suffices -- the producer only overwrites cells below this index
       if (rd && ch.in_ring && lead && (((t0 >> 2) & 1) || t0 + 4 >= T))
-        st_relaxed_cluster(ch.in_cons, ch.in_base + min(t0 + 4 + ioff, T));
+        st_relaxed_cta(ch.in_cons, ch.in_base + min(t0 + 4 + ioff, T));
     }
   }
   if constexpr (LINKED) {
-    if (rd && ch.in_ring && lead) st_relaxed_cluster(ch.in_cons, ch.in_base + T);  // everything consumed
+    if (rd && ch.in_ring && lead) st_relaxed_cta(ch.in_cons, ch.in_base + T);  // everything consumed
   }
 }
 
@@ -590,18 +498,11 @@ __device__ __forceinline__ void short_item(const ShortArgs& a, int item, uint8_t
 // current strip ends) through a global row per CTA.  A pair never spans CTAs:
 // every wait is on a warp of the same CTA, so nothing depends on co-residency.
 struct LongShared {
-  int prog[LONG_W];          // per local consumer warp: its producer's progress
-  int cons[LONG_W];          // per local producer warp: its consumer's consumption
-  int wprog;                 // round-wrap progress (the CTA holding position 0)
-  int item;                  // the cluster's current item (CTA rank 0's copy is the one read)
-  int pbest[2 * LONG_W * 4]; // per pair of the item: max of each s16x2 half (CTA rank 0's copy)
+  int prog[LONG_W];
+  int cons[LONG_W];
+  uint32_t best[LONG_W];
 };
 
-// One long item on the KC CTAs of a thread-block cluster (KC = 1 without a
-// cluster launch): TW = KC x LONG_W warps chain the strips of one pair (or of
-// `pack` pairs side by side when the query has fewer strips than TW).  All CTAs
-// of a cluster are co-scheduled, so warps of different CTAs may wait on each
-// other across rounds (the round wrap) without any co-residency assumption.
 template <bool NIB>
 __device__ __forceinline__ void long_item(const LongArgs& a, int item, uint8_t* smem, LongShared& sh) {
   constexpr int W = LONG_W;
@@ -609,103 +510,95 @@ __device__ __forceinline__ void long_item(const LongArgs& a, int item, uint8_t* 
   // consumption; the consumer starts only once the producer is ioff + 4 +
   // LINK_LAG steps in, so the ring must hold more than that (else both wait).
   static_assert(LONG_RING - 4 >= (32 * SubLanes<LONG_R>::V - 1) + 4 + LINK_LAG + 16, "ring too short for the lag");
-  uint2* rings = reinterpret_cast<uint2*>(smem);                       // [W][LONG_RING], per local consumer warp
-  uint8_t* lprof = smem + W * LONG_RING * sizeof(uint2);               // [W][SBL]
+  uint2* rings = reinterpret_cast<uint2*>(smem);                       // [W - 1][LONG_RING]
+  uint8_t* lprof = smem + (W - 1) * LONG_RING * sizeof(uint2);         // [W][SBL]
+  int* s_prog = sh.prog;
+  int* s_cons = sh.cons;
+  uint32_t* s_best = sh.best;
   const int tid = threadIdx.x;
   const int lane = tid & 31, warp = tid >> 5;
-  const uint32_t KC = cluster_nctarank(), crank = cluster_ctarank();
-  auto csync = [&]() { if (KC > 1) cluster_sync_all(); else __syncthreads(); };
-  const int TW = int(KC) * W;                    // warps of the cluster
-  const int gw = int(crank) * W + warp;          // this warp's index in the cluster
-  uint2* wrap = a.wrap + (size_t)(blockIdx.x / KC) * a.wcap;
-  if (tid < W) { sh.prog[tid] = -1; sh.cons[tid] = 0; }
-  if (tid == 0) sh.wprog = -1;
-  for (int i = tid; i < W * LONG_RING; i += blockDim.x)  // every cell "written in lap -1"
-    rings[i] = make_uint2(0x80008000u, 0u);
-  if (crank == 0)
-    for (int i = tid; i < 2 * W * 4; i += blockDim.x) sh.pbest[i] = 0;
-  csync();  // every CTA reset before any remote write of this item
-  const int2 li = a.lmap[item];  // (query, item within the query), costliest first across queries
-  const LongQuery d = a.queries[li.x];
-  const int ns = d.n_strips;
-  // a query of fewer strips than the cluster's warps: P (host-chosen) pairs per item, ns warps each
-  const int P = d.pack;
-  const int GS = ns >= TW ? TW : ns;             // warps per pair
-  const int grp = gw / GS, wg = gw - grp * GS;
-  const int j = GS - 1 - wg;                     // position of this warp's strip within a round
-  const int pidx = li.y * P + grp;
-  const bool active = grp < P && pidx < d.n_long;
-  PairRec pr;
-  if (active) pr = a.pairs[pidx];
-  else { pr.off = 0; pr.len = 0; pr.id0 = -1; pr.id1 = -1; }
-  constexpr int VG = 32 * SubLanes<LONG_R>::V;
-  const int T = pr.len + VG;
-  uint32_t best = 0;
-  uint8_t* myprof = lprof + warp * a.SBL;
-  // neighbours: position j-1 (producer) is warp gw+1, position j+1 (consumer) is warp gw-1;
-  // the round wrap: position GS-1 (warp grp*GS) -> position 0 (warp grp*GS + GS-1)
-  const int gprod = gw + 1, gcons = gw - 1, gz = grp * GS + GS - 1;
-  for (int r = 0; active; ++r) {
-    const int s = GS * r + j;  // strip index
-    if (s >= ns) break;
-    __syncwarp();
-    {  // this warp's strip profile -> its own slot
-      const uint4* src = reinterpret_cast<const uint4*>(d.prof_long + (size_t)s * a.SBL);
-      uint4* dst = reinterpret_cast<uint4*>(myprof);
-      for (int i = lane; i < a.SBL / 16; i += 32) dst[i] = __ldg(src + i);
+  uint2* wrap = a.wrap + (size_t)blockIdx.x * a.wcap;
+  {
+    if (tid < W) { s_prog[tid] = -1; s_cons[tid] = 0; s_best[tid] = 0; }
+    __syncthreads();
+    const int2 li = a.lmap[item];  // (query, item within the query), costliest first across queries
+    const LongQuery d = a.queries[li.x];
+    const int ns = d.n_strips;
+    // a query of fewer strips than warps: P (host-chosen, <= W / ns) pairs per item, ns warps each
+    const int P = d.pack;
+    const int GS = ns >= W ? W : ns;             // warps per pair
+    const int grp = warp / GS, wg = warp - grp * GS;
+    const int j = GS - 1 - wg;                   // position of this warp's strip within a round
+    const int pidx = li.y * P + grp;
+    const bool active = grp < P && pidx < d.n_long;
+    PairRec pr;
+    if (active) pr = a.pairs[pidx];
+    else { pr.off = 0; pr.len = 0; pr.id0 = -1; pr.id1 = -1; }
+    constexpr int VG = 32 * SubLanes<LONG_R>::V;
+    const int T = pr.len + VG;
+    uint32_t best = 0;
+    uint8_t* myprof = lprof + warp * a.SBL;
+    const int lbase = grp * (GS - 1), cbase = grp * GS;  // this pair's rings and counters
+    for (int r = 0; active; ++r) {
+      const int s = GS * r + j;  // strip index
+      if (s >= ns) break;
+      __syncwarp();
+      {  // this warp's strip profile -> its own slot
+        const uint4* src = reinterpret_cast<const uint4*>(d.prof_long + (size_t)s * a.SBL);
+        uint4* dst = reinterpret_cast<uint4*>(myprof);
+        for (int i = lane; i < a.SBL / 16; i += 32) dst[i] = __ldg(src + i);
+      }
+      __syncwarp();
+      const bool rd = s > 0, wr = s + 1 < ns;
+      Chain ch{};
+      ch.out_base = r * T;
+      // input: ring j-1 (same round) or the wrap row (previous round, from position GS-1)
+      ch.in_ring = j > 0;
+      if (j > 0) {
+        ch.in_sring = static_cast<uint32_t>(__cvta_generic_to_shared(rings + (size_t)(lbase + j - 1) * LONG_RING));
+        ch.in_prog = &s_prog[cbase + j - 1];
+        ch.in_cons = &s_cons[cbase + j - 1];
+        ch.in_base = r * T;
+      } else {
+        ch.in_prog = &s_prog[cbase + GS - 1];
+        ch.grow_in = wrap;
+        ch.in_base = (r - 1) * T;   // the wrap row was written in the previous round
+      }
+      ch.out_ring = j < GS - 1;
+      if (j < GS - 1) {
+        ch.out_sring = static_cast<uint32_t>(__cvta_generic_to_shared(rings + (size_t)(lbase + j) * LONG_RING));
+        ch.out_cons = &s_cons[cbase + j];
+      } else {
+        ch.grow_out = wrap;         // only reached when ns > W (P = 1): the round wrap
+      }
+      ch.out_prog = &s_prog[cbase + j];
+      const void* pstream = NIB ? static_cast<const void*>(reinterpret_cast<const uint8_t*>(a.stream) + pr.off)
+                                : static_cast<const void*>(a.stream + pr.off);
+      strip_pass<32, LONG_R, true, false, LONG_US, NIB>(myprof, a.LSL, a.LBL, pstream, pr.len, T, lane, rd, wr,
+                                                   nullptr, nullptr, ch, a.code_pad2, a.nGe, a.nGsGe, best);
     }
-    __syncwarp();
-    const bool rd = s > 0, wr = s + 1 < ns;
-    Chain ch{};
-    ch.cluster = KC > 1;
-    ch.out_base = r * T;
-    ch.in_ring = j > 0;
-    if (j > 0) {  // input: ring of the producer warp (same round), held here
-      ch.in_sring = static_cast<uint32_t>(__cvta_generic_to_shared(rings + (size_t)warp * LONG_RING));
-      ch.in_cons = map_rank(&sh.cons[gprod % W], uint32_t(gprod / W));
-      ch.in_base = r * T;
-    } else {      // input: the wrap row of the previous round
-      ch.in_prog = &sh.wprog;
-      ch.grow_in = wrap;
-      ch.in_base = (r - 1) * T;
-    }
-    ch.out_ring = j < GS - 1;
-    if (j < GS - 1) {
-      ch.out_ring_ptr = map_rank(rings + (size_t)(gcons % W) * LONG_RING, uint32_t(gcons / W));
-      ch.out_cons = &sh.cons[warp];
-    } else {      // only reached when ns > TW (P = 1): the round wrap
-      ch.grow_out = wrap;
-      ch.out_prog = map_rank(&sh.wprog, uint32_t(gz / W));
-    }
-    const void* pstream = NIB ? static_cast<const void*>(reinterpret_cast<const uint8_t*>(a.stream) + pr.off)
-                              : static_cast<const void*>(a.stream + pr.off);
-    strip_pass<32, LONG_R, true, false, LONG_US, NIB>(myprof, a.LSL, a.LBL, pstream, pr.len, T, lane, rd, wr,
-                                                     nullptr, nullptr, ch, a.code_pad2, a.nGe, a.nGsGe, best);
-  }
 #pragma unroll
-  for (int o = 16; o > 0; o >>= 1) best = __vmaxs2(best, __shfl_xor_sync(FULL, best, o));
-  if (lane == 0 && active) {
-    int* pb = map_rank(&sh.pbest[2 * grp], 0u);
-    atomicMax(pb, int(int16_t(best & 0xffffu)));
-    atomicMax(pb + 1, int(int16_t(best >> 16)));
-  }
-  csync();
-  if (crank == 0 && tid < P) {
-    const int pj = li.y * P + tid;
-    if (pj < d.n_long) {
-      const PairRec pq = a.pairs[pj];
-      const int v0 = sh.pbest[2 * tid], v1 = sh.pbest[2 * tid + 1];
-      d.scores[pq.id0] = v0;
-      if (v0 >= a.thr) flag_overflow(a.ovf_count, a.ovf, a.ovf_cap, d.qidx, pj, 0);
-      if (pq.id1 >= 0) {
-        d.scores[pq.id1] = v1;
-        if (v1 >= a.thr) flag_overflow(a.ovf_count, a.ovf, a.ovf_cap, d.qidx, pj, 1);
+    for (int o = 16; o > 0; o >>= 1) best = __vmaxs2(best, __shfl_xor_sync(FULL, best, o));
+    if (lane == 0) s_best[warp] = best;
+    __syncthreads();
+    if (tid < P) {
+      const int pj = li.y * P + tid;
+      if (pj < d.n_long) {
+        const PairRec pq = a.pairs[pj];
+        uint32_t b = 0;
+        for (int w = tid * GS; w < tid * GS + GS; ++w) b = __vmaxs2(b, s_best[w]);
+        const int v0 = int(int16_t(b & 0xffffu)), v1 = int(int16_t(b >> 16));
+        d.scores[pq.id0] = v0;
+        if (v0 >= a.thr) flag_overflow(a.ovf_count, a.ovf, a.ovf_cap, d.qidx, pj, 0);
+        if (pq.id1 >= 0) {
+          d.scores[pq.id1] = v1;
+          if (v1 >= a.thr) flag_overflow(a.ovf_count, a.ovf, a.ovf_cap, d.qidx, pj, 1);
+        }
       }
     }
+    __syncthreads();
   }
-  csync();
 }
-
 // The short-pair kernel: one persistent launch per short-pair mode (query pairs,
 // single query), one (G, R) per launch, its own register budget (the query-pair
 // form keeps R = 32 rows per lane at 128 registers, 2 CTAs per SM).
@@ -772,16 +665,15 @@ __global__ void __launch_bounds__(NT, 2) combined_m0_kernel(ShortArgs as, LongAr
 template <bool NIB>
 __global__ void __launch_bounds__(LONG_W * 32, 2) long_kernel(LongArgs al) {
   extern __shared__ __align__(128) uint8_t smem[];
+  __shared__ int s_item;
   __shared__ LongShared sh;
-  const uint32_t KC = cluster_nctarank(), crank = cluster_ctarank();
-  for (;;) {  // the cluster takes one item at a time (CTA rank 0 fetches, the others read its copy)
-    if (crank == 0 && threadIdx.x == 0) sh.item = atomicAdd(al.work_counter, 1);
-    if (KC > 1) cluster_sync_all(); else __syncthreads();
-    const int item = *map_rank(&sh.item, 0u);
-    // every CTA has read the item before CTA 0 may exit (its shared memory would vanish)
-    if (KC > 1) cluster_sync_all(); else __syncthreads();
+  for (;;) {
+    if (threadIdx.x == 0) s_item = atomicAdd(al.work_counter, 1);
+    __syncthreads();
+    const int item = s_item;
+    __syncthreads();
     if (item >= al.n_items) break;
-    long_item<NIB>(al, item, smem, sh);  // ends with a cluster barrier: sh.item may be rewritten
+    long_item<NIB>(al, item, smem, sh);
   }
 }
 
@@ -910,50 +802,19 @@ cudaError_t launch_combined(int G, int R, int grid, int smem_bytes, const ShortA
   return cudaGetLastError();
 }
 
-// Resident clusters of kc CTAs (kc = 1: resident CTAs), for sizing the persistent grid.
-int long_max_clusters(int smem_bytes, bool nib, int kc) {
-  auto f = nib ? long_kernel<true> : long_kernel<false>;
-  if (smem_bytes > 48 * 1024) cudaFuncSetAttribute(f, cudaFuncAttributeMaxDynamicSharedMemorySize, smem_bytes);
-  if (kc <= 1) return occupancy(reinterpret_cast<const void*>(f), LONG_W * 32, smem_bytes);
-  cudaLaunchConfig_t cfg{};
-  cfg.gridDim = dim3(unsigned(kc) * 148u, 1, 1);
-  cfg.blockDim = dim3(LONG_W * 32, 1, 1);
-  cfg.dynamicSmemBytes = size_t(smem_bytes);
-  cudaLaunchAttribute at[1];
-  at[0].id = cudaLaunchAttributeClusterDimension;
-  at[0].val.clusterDim.x = unsigned(kc);
-  at[0].val.clusterDim.y = 1;
-  at[0].val.clusterDim.z = 1;
-  cfg.attrs = at;
-  cfg.numAttrs = 1;
-  int n = 0;
-  if (cudaOccupancyMaxActiveClusters(&n, reinterpret_cast<const void*>(f), &cfg) != cudaSuccess) return 0;
-  return n;
+int long_max_ctas_per_sm(int smem_bytes, bool nib) {
+  return occupancy(nib ? reinterpret_cast<const void*>(long_kernel<true>) : reinterpret_cast<const void*>(long_kernel<false>),
+                   LONG_W * 32, smem_bytes);
 }
 
-cudaError_t launch_long(int grid, int smem_bytes, const LongArgs& a, cudaStream_t st, bool nib, int kc) {
+cudaError_t launch_long(int grid, int smem_bytes, const LongArgs& a, cudaStream_t st, bool nib) {
   auto f = nib ? long_kernel<true> : long_kernel<false>;
   if (smem_bytes > 48 * 1024) {
     cudaError_t e = cudaFuncSetAttribute(f, cudaFuncAttributeMaxDynamicSharedMemorySize, smem_bytes);
     if (e != cudaSuccess) return e;
   }
-  if (kc <= 1) {
-    f<<<grid, LONG_W * 32, smem_bytes, st>>>(a);
-    return cudaGetLastError();
-  }
-  cudaLaunchConfig_t cfg{};
-  cfg.gridDim = dim3(unsigned(grid), 1, 1);
-  cfg.blockDim = dim3(LONG_W * 32, 1, 1);
-  cfg.dynamicSmemBytes = size_t(smem_bytes);
-  cfg.stream = st;
-  cudaLaunchAttribute at[1];
-  at[0].id = cudaLaunchAttributeClusterDimension;
-  at[0].val.clusterDim.x = unsigned(kc);
-  at[0].val.clusterDim.y = 1;
-  at[0].val.clusterDim.z = 1;
-  cfg.attrs = at;
-  cfg.numAttrs = 1;
-  return cudaLaunchKernelEx(&cfg, f, a);
+  f<<<grid, LONG_W * 32, smem_bytes, st>>>(a);
+  return cudaGetLastError();
 }
 
 // ---------------------------------------------------------------------------

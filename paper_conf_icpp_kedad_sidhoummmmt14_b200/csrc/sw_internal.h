@@ -60,10 +60,7 @@ struct ProfGeom {
 // 16 lanes of an LDS.64 phase hit 16 distinct 8-byte slots whatever letters they read)
 constexpr int LONG_R = 16;
 constexpr int LONG_US = 32 * 8;     // bytes between a lane's consecutive 8-byte units in the long profile
-#ifndef SW_LONG_RING
-#define SW_LONG_RING 128
-#endif
-constexpr int LONG_RING = SW_LONG_RING;  // steps held by a shared-memory link ring between two warps of a CTA
+constexpr int LONG_RING = 128;      // steps held by a shared-memory link ring between two warps of a CTA
 
 // Long (intra-task) work of one query: pairs [0, n_long) of the DB are scored by
 // the chained warps of one CTA each.
@@ -201,9 +198,8 @@ int short_max_ctas_per_sm(int mode, int G, int R, int smem_bytes, bool cg = fals
                           int nt = SCORE_NT);
 cudaError_t launch_short(int mode, int G, int R, int grid, int smem_bytes, const ShortArgs& a, cudaStream_t st,
                          bool cg = false, bool nib = false, int nt = SCORE_NT);
-// kc: CTAs per thread-block cluster of the long kernel (one long item per cluster)
-int long_max_clusters(int smem_bytes, bool nib, int kc);
-cudaError_t launch_long(int grid, int smem_bytes, const LongArgs& a, cudaStream_t st, bool nib, int kc);
+int long_max_ctas_per_sm(int smem_bytes, bool nib = false);
+cudaError_t launch_long(int grid, int smem_bytes, const LongArgs& a, cudaStream_t st, bool nib = false);
 // single-query searches with long pairs: long items and mode-0 short items in one launch
 int combined_max_ctas_per_sm(int G, int R, int smem_bytes, bool nib = false);
 cudaError_t launch_combined(int G, int R, int grid, int smem_bytes, const ShortArgs& as, const LongArgs& al,

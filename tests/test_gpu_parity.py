@@ -525,17 +525,15 @@ def test_small_search_one_group_ctas(small):
         np.testing.assert_array_equal(got, oracle_scores(qc, qo, dc, do))
 
 
-@pytest.mark.parametrize("cluster", [1, 0])
-def test_long_only_search_on_clusters(cluster):
+def test_long_only_search_tall_queries():
     """A search whose pairs are all long (every DB sequence longer than t_long)
-    runs the long kernel alone; tall queries split each pair over a thread-block
-    cluster (2 CTAs for 26 strips, 3 for 69: the strips chain across CTAs through
-    distributed shared memory, the round wrap through global memory); queries of
-    fewer strips than the cluster's warps pack several pairs per item.  Option
-    long_cluster 0: one CTA per pair.  Both equal the oracle."""
-    rng = np.random.default_rng(240 + cluster)
+    runs the long kernel alone: tall queries (26 and 69 strips) chain their
+    strips over the warps of one CTA in rounds (the round wrap through global
+    memory); queries of fewer strips than the CTA's warps pack several pairs per
+    item.  Equals the oracle."""
+    rng = np.random.default_rng(240)
     dc, do = _seqs(list(rng.integers(70, 900, size=24)) + [3001, 1500], rng)
     for ql in ([13000, 100, 700], [35000, 2000]):
         qc, qo = _seqs(ql, rng)
-        got = gpu_scores(qc, qo, dc, do, opts={"t_long": 64, "long_cluster": cluster})
+        got = gpu_scores(qc, qo, dc, do, opts={"t_long": 64})
         np.testing.assert_array_equal(got, oracle_scores(qc, qo, dc, do, procs=16))

@@ -75,7 +75,6 @@ struct SwError {
 [[noreturn]] void fail(int32_t code, const std::string& m) { throw SwError{code, m}; }
 
 constexpr int T_LONG = 3000;
-constexpr int LONG_ROUNDS = 3;  // target rounds of W strips per CTA for a long pair
 // A short item (one lane group, all strips of its query) may run at most
 // max(CRIT_MIN_STEPS, CRIT_FRACTION x the average lane group's wavefront steps
 // of the launch); longer (query, pair) work goes to the intra-task mode.
@@ -724,6 +723,7 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
   struct LItem { double cost; int q, it; };
   std::vector<LItem> litems;
   int64_t long_items = 0;
+  int wrap_groups = 1;  // pair groups per CTA that need a round-wrap row
   int32_t max_long = 0;
   for (size_t k = 0; k < order.size(); ++k) {
     const int nl = qnlong[k];
@@ -736,10 +736,31 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
     d.n_strips = gl[k].n_strips;
     d.qidx = order[k];
     d.n_long = nl;
-    d.pack = (combined || gl[k].n_strips >= W) ? 1 : W / gl[k].n_strips;
+    // warps per pair GS and pairs per item P (P * GS <= W): the fewest idle warp-rounds
+    // (ns strips over GS warps take ceil(ns / GS) rounds; W - P * GS warps idle), ties to
+    // the larger GS (fewer rounds: a shorter critical path per item); at most
+    // max(ceil(ns / W), 5) rounds.  The combined
+    // single-query launch keeps one pair per item.
+    const int ns = gl[k].n_strips;
+#ifndef SW_COMBINED_PACK
+#define SW_COMBINED_PACK 0
+#endif
+    const bool one_pair = combined && !SW_COMBINED_PACK;
+    int GS = std::min(ns, W), P = one_pair ? 1 : W / GS;
+    if (!one_pair) {
+      double best_eff = -1;
+      for (int g = std::min(ns, W); g >= 1; --g) {
+        const int p = W / g, rr = (ns + g - 1) / g;
+        if (rr > std::max((ns + W - 1) / W, 5)) continue;  // bounds the item's critical path
+        const double eff = double(p) * ns / (double(W) * rr);
+        if (eff > best_eff + 1e-9) { best_eff = eff; GS = g; P = p; }
+      }
+    }
+    d.pack = P;
+    d.gs = GS;
+    if (ns > GS) wrap_groups = std::max(wrap_groups, P);
     // item cost: rounds x the item's longest pair (pairs are sorted longest first)
-    const int GS = gl[k].n_strips >= W ? W : gl[k].n_strips;
-    const double rounds = double((gl[k].n_strips + GS - 1) / GS);
+    const double rounds = double((ns + GS - 1) / GS);
     for (int it = 0; it * d.pack < nl; ++it)
       litems.push_back({rounds * double(db->pairs[size_t(it * d.pack)].len + 64), int(ldesc.size()), it});
     ldesc.push_back(d);
@@ -911,7 +932,8 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
     const int occ = long_max_ctas_per_sm(smem, nib);
     if (occ <= 0) fail(SW_ECUDA, "long-pair kernel does not fit on an SM");
     const int grid = int(std::max<int64_t>(1, std::min<int64_t>(long_items, int64_t(occ) * h->sms)));
-    SW_CK(h->wrap.ensure(size_t(grid) * al.wcap * sizeof(uint2)));
+    al.wrap_groups = wrap_groups;
+    SW_CK(h->wrap.ensure(size_t(grid) * wrap_groups * al.wcap * sizeof(uint2)));
     al.wrap = h->wrap.as<uint2>();
     cudaStream_t lst = c.st;
     if (fork) {
@@ -991,7 +1013,8 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
     std::pair<cudaEvent_t, cudaEvent_t>* ev = nullptr;
     record_begin(h, c.timing, 0, c.st, ev);
     if (with_long) {
-      SW_CK(h->wrap.ensure(size_t(grid) * al.wcap * sizeof(uint2)));
+      al.wrap_groups = wrap_groups;
+      SW_CK(h->wrap.ensure(size_t(grid) * wrap_groups * al.wcap * sizeof(uint2)));
       al.wrap = h->wrap.as<uint2>();
       SW_CK(launch_combined(G, R, grid, smem, as, al, c.st, nib));
     } else {

@@ -517,17 +517,17 @@ __device__ __forceinline__ void long_item(const LongArgs& a, int item, uint8_t* 
   uint32_t* s_best = sh.best;
   const int tid = threadIdx.x;
   const int lane = tid & 31, warp = tid >> 5;
-  uint2* wrap = a.wrap + (size_t)blockIdx.x * a.wcap;
   {
     if (tid < W) { s_prog[tid] = -1; s_cons[tid] = 0; s_best[tid] = 0; }
     __syncthreads();
     const int2 li = a.lmap[item];  // (query, item within the query), costliest first across queries
     const LongQuery d = a.queries[li.x];
     const int ns = d.n_strips;
-    // a query of fewer strips than warps: P (host-chosen, <= W / ns) pairs per item, ns warps each
+    // P pairs per item, GS warps each (host-chosen, P * GS <= W: few idle warp-rounds)
     const int P = d.pack;
-    const int GS = ns >= W ? W : ns;             // warps per pair
+    const int GS = d.gs;
     const int grp = warp / GS, wg = warp - grp * GS;
+    uint2* wrap = a.wrap + ((size_t)blockIdx.x * a.wrap_groups + (grp < a.wrap_groups ? grp : 0)) * a.wcap;
     const int j = GS - 1 - wg;                   // position of this warp's strip within a round
     const int pidx = li.y * P + grp;
     const bool active = grp < P && pidx < d.n_long;
@@ -569,7 +569,7 @@ __device__ __forceinline__ void long_item(const LongArgs& a, int item, uint8_t* 
         ch.out_sring = static_cast<uint32_t>(__cvta_generic_to_shared(rings + (size_t)(lbase + j) * LONG_RING));
         ch.out_cons = &s_cons[cbase + j];
       } else {
-        ch.grow_out = wrap;         // only reached when ns > W (P = 1): the round wrap
+        ch.grow_out = wrap;         // only reached when ns > GS: the round wrap
       }
       ch.out_prog = &s_prog[cbase + j];
       const void* pstream = NIB ? static_cast<const void*>(reinterpret_cast<const uint8_t*>(a.stream) + pr.off)

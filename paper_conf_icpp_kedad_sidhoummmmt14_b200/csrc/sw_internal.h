@@ -70,8 +70,9 @@ struct LongQuery {
   int n_strips;
   int qidx;
   int n_long;
-  int pack;                  // pairs per item: 1, or up to W / n_strips when n_strips < W (the
-                             // CTA's warps then chain several pairs side by side)
+  int pack;                  // pairs per item (P): the CTA's warps chain P pairs side by side
+  int gs;                    // warps per pair (GS, P * GS <= W): a pair's strips go round-robin
+                             // over its GS warps, ceil(n_strips / GS) rounds
 };
 
 struct LongArgs {
@@ -80,7 +81,9 @@ struct LongArgs {
   int n_items;               // long items of the launch
   const int2* lmap;          // item -> (query, item within the query), costliest first
   int SBL, LSL, LBL;         // long profile geometry
-  uint2* wrap;               // [gridDim][wcap]: the round-wrap link row of each CTA (warp W-1 -> warp 0)
+  uint2* wrap;               // [gridDim][wrap_groups][wcap]: the round-wrap link row of each pair
+                             // group of a CTA (its last warp -> its first warp, next round)
+  int wrap_groups;           // max pairs per item among queries of more strips than warps per pair
   int wcap;
   const uint16_t* stream;
   const PairRec* pairs;

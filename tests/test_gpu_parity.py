@@ -533,7 +533,9 @@ def test_long_only_search_tall_queries():
     item.  Equals the oracle."""
     rng = np.random.default_rng(240)
     dc, do = _seqs(list(rng.integers(70, 900, size=24)) + [3001, 1500], rng)
-    for ql in ([13000, 100, 700], [35000, 2000]):
+    # 26 / 69 strips: 8 warps per pair; 4 strips: 2 pairs of 4 warps; 10 strips: 4 pairs of
+    # 2 warps (5 rounds, one round-wrap row per pair group); 20 strips: 2 pairs of 4 warps
+    for ql in ([13000, 100, 700], [35000, 2000], [5000, 10000, 300]):
         qc, qo = _seqs(ql, rng)
         got = gpu_scores(qc, qo, dc, do, opts={"t_long": 64})
         np.testing.assert_array_equal(got, oracle_scores(qc, qo, dc, do, procs=16))

@@ -59,6 +59,72 @@ struct DevBuf {
   template <class T> T* as() const { return reinterpret_cast<T*>(p); }
 };
 
+// Pinned staging of a search's host -> device uploads (queries, work-item tables).
+// A cudaMemcpyAsync from pageable memory first waits for the stream to drain, so a
+// search's host-side preparation would run while the GPU idles; from pinned memory
+// the copies queue behind the previous search's kernels.  Two halves alternate
+// between consecutive searches; a half is refilled only after the event recorded
+// behind its last copy (two searches ago) has completed.
+struct HostStage {
+  struct Half {
+    uint8_t* p = nullptr;
+    size_t cap = 0, used = 0;
+    cudaEvent_t ev = nullptr;
+    bool pending = false;
+    std::vector<uint8_t*> retired;  // outgrown buffers, freed once `ev` completes
+  };
+  Half half[2];
+  int cur = 0;
+  cudaError_t begin() {
+    cur ^= 1;
+    Half& H = half[cur];
+    if (H.pending) {
+      cudaError_t e = cudaEventSynchronize(H.ev);
+      if (e != cudaSuccess) return e;
+      H.pending = false;
+    }
+    for (uint8_t* q : H.retired) cudaFreeHost(q);
+    H.retired.clear();
+    H.used = 0;
+    return cudaSuccess;
+  }
+  cudaError_t copy(void* dst, const void* src, size_t bytes, cudaStream_t st) {
+    if (bytes == 0) return cudaSuccess;
+    Half& H = half[cur];
+    size_t off = (H.used + 15) & ~size_t(15);
+    if (off + bytes > H.cap) {  // grow: earlier copies of this search may still read the old buffer
+      const size_t cap = std::max<size_t>({2 * H.cap, off + bytes, size_t(1) << 20});
+      uint8_t* q = nullptr;
+      cudaError_t e = cudaMallocHost(&q, cap);
+      if (e != cudaSuccess) return e;
+      if (H.p) H.retired.push_back(H.p);
+      H.p = q;
+      H.cap = cap;
+      off = 0;
+    }
+    if (!H.ev) {
+      cudaError_t e = cudaEventCreateWithFlags(&H.ev, cudaEventDisableTiming);
+      if (e != cudaSuccess) return e;
+    }
+    std::memcpy(H.p + off, src, bytes);
+    H.used = off + bytes;
+    cudaError_t e = cudaMemcpyAsync(dst, H.p + off, bytes, cudaMemcpyHostToDevice, st);
+    if (e != cudaSuccess) return e;
+    H.pending = true;
+    return cudaEventRecord(H.ev, st);  // behind every copy: an early exit never leaves one unguarded
+  }
+  void release() {
+    for (Half& H : half) {
+      if (H.pending && H.ev) cudaEventSynchronize(H.ev);
+      for (uint8_t* q : H.retired) cudaFreeHost(q);
+      H.retired.clear();
+      if (H.p) cudaFreeHost(H.p);
+      if (H.ev) cudaEventDestroy(H.ev);
+      H = Half{};
+    }
+  }
+};
+
 struct SwError {
   int32_t code;
   std::string msg;
@@ -99,6 +165,7 @@ struct sw_handle_s {
   DevBuf imap;            // short work item order (mode 1 items, then mode 0 items)
   DevBuf lmap;            // long work item order
   DevBuf vq, sinfo;       // packed mode-1 slots: strip-padded query codes per half, per-strip info
+  HostStage stage;        // pinned staging of sw_search's uploads
   cudaStream_t side = nullptr;             // the long-pair kernel's stream when short pairs run too
   cudaEvent_t ev_fork = nullptr, ev_join = nullptr;
 
@@ -742,12 +809,8 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
     // max(ceil(ns / W), 5) rounds.  The combined
     // single-query launch keeps one pair per item.
     const int ns = gl[k].n_strips;
-#ifndef SW_COMBINED_PACK
-#define SW_COMBINED_PACK 0
-#endif
-    const bool one_pair = combined && !SW_COMBINED_PACK;
-    int GS = std::min(ns, W), P = one_pair ? 1 : W / GS;
-    if (!one_pair) {
+    int GS = std::min(ns, W), P = combined ? 1 : W / GS;
+    if (!combined) {
       double best_eff = -1;
       for (int g = std::min(ns, W); g >= 1; --g) {
         const int p = W / g, rr = (ns + g - 1) / g;
@@ -874,23 +937,23 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
   }
   if (long_items + int64_t(imap.size()) >= (int64_t(1) << 31)) fail(SW_EUNSUPPORTED, "too many work items");
   if (si_total)
-    SW_CK(cudaMemcpyAsync(h->sinfo.p, sinfo.data(), si_total * sizeof(StripInfo), cudaMemcpyHostToDevice, c.st));
+    SW_CK(h->stage.copy(h->sinfo.p, sinfo.data(), si_total * sizeof(StripInfo), c.st));
   SW_CK(h->imap.ensure(std::max<size_t>(imap.size(), 1) * sizeof(int2)));
   if (!imap.empty())
-    SW_CK(cudaMemcpyAsync(h->imap.p, imap.data(), imap.size() * sizeof(int2), cudaMemcpyHostToDevice, c.st));
+    SW_CK(h->stage.copy(h->imap.p, imap.data(), imap.size() * sizeof(int2), c.st));
   // long items costliest first across all queries (so no big item starts late)
   std::stable_sort(litems.begin(), litems.end(), [](const LItem& x, const LItem& y) { return x.cost > y.cost; });
   std::vector<int2> lmap(litems.size());
   for (size_t i = 0; i < litems.size(); ++i) lmap[i] = make_int2(litems[i].q, litems[i].it);
   SW_CK(h->lmap.ensure(std::max<size_t>(lmap.size(), 1) * sizeof(int2)));
   if (!lmap.empty())
-    SW_CK(cudaMemcpyAsync(h->lmap.p, lmap.data(), lmap.size() * sizeof(int2), cudaMemcpyHostToDevice, c.st));
+    SW_CK(h->stage.copy(h->lmap.p, lmap.data(), lmap.size() * sizeof(int2), c.st));
   SW_CK(h->qdesc.ensure(ldesc.size() * sizeof(LongQuery) + sdesc.size() * sizeof(SlotDesc) + 16));
   LongQuery* d_ldesc = h->qdesc.as<LongQuery>();
   SlotDesc* d_slots = reinterpret_cast<SlotDesc*>(h->qdesc.as<uint8_t>() + ldesc.size() * sizeof(LongQuery));
   if (!ldesc.empty())
-    SW_CK(cudaMemcpyAsync(d_ldesc, ldesc.data(), ldesc.size() * sizeof(LongQuery), cudaMemcpyHostToDevice, c.st));
-  SW_CK(cudaMemcpyAsync(d_slots, sdesc.data(), sdesc.size() * sizeof(SlotDesc), cudaMemcpyHostToDevice, c.st));
+    SW_CK(h->stage.copy(d_ldesc, ldesc.data(), ldesc.size() * sizeof(LongQuery), c.st));
+  SW_CK(h->stage.copy(d_slots, sdesc.data(), sdesc.size() * sizeof(SlotDesc), c.st));
   SW_CK(h->counters.ensure(3 * sizeof(int)));
   SW_CK(cudaMemsetAsync(h->counters.p, 0, 3 * sizeof(int), c.st));
   int* counters = h->counters.as<int>();
@@ -1097,9 +1160,10 @@ int32_t sw_search(sw_handle_t h, const uint8_t* q_codes, const int64_t* q_offset
     SW_CK(h->qcodes.ensure(size_t(std::max<int64_t>(qtot, 1))));
     SW_CK(h->qoff.ensure(qoff0.size() * sizeof(int64_t)));
     SW_CK(h->matrix.ensure(size_t(alpha * alpha)));
-    if (qtot) SW_CK(cudaMemcpyAsync(h->qcodes.p, qbase, size_t(qtot), cudaMemcpyHostToDevice, st));
-    SW_CK(cudaMemcpyAsync(h->qoff.p, qoff0.data(), qoff0.size() * sizeof(int64_t), cudaMemcpyHostToDevice, st));
-    SW_CK(cudaMemcpyAsync(h->matrix.p, matrix, size_t(alpha * alpha), cudaMemcpyHostToDevice, st));
+    SW_CK(h->stage.begin());
+    SW_CK(h->stage.copy(h->qcodes.p, qbase, size_t(qtot), st));
+    SW_CK(h->stage.copy(h->qoff.p, qoff0.data(), qoff0.size() * sizeof(int64_t), st));
+    SW_CK(h->stage.copy(h->matrix.p, matrix, size_t(alpha * alpha), st));
     int launches = 0;
     if (!db->mapped) {
       SW_CK(cudaMemsetAsync(dscores, 0, out_bytes, st));
@@ -1544,6 +1608,7 @@ int32_t sw_free(sw_handle_t h) {
     if (e) cudaEventDestroy(e);
   if (h->side) cudaStreamDestroy(h->side);
   if (h->ev_done) cudaEventDestroy(h->ev_done);
+  h->stage.release();
   delete h;
   return SW_OK;
 }

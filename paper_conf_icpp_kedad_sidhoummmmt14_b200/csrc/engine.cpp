@@ -145,6 +145,7 @@ constexpr int T_LONG = 3000;
 // max(CRIT_MIN_STEPS, CRIT_FRACTION x the average lane group's wavefront steps
 // of the launch); longer (query, pair) work goes to the intra-task mode.
 constexpr int64_t CRIT_MIN_STEPS = 16384;
+constexpr double LINK_LAG_STEPS = 32;   // the long kernel's producer lead (kernels.cu LINK_LAG)
 constexpr double CRIT_FRACTION = 0.35;  // pairs longer than this are launched separately
 
 }  // namespace
@@ -792,6 +793,43 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
   int64_t long_items = 0;
   int wrap_groups = 1;  // pair groups per CTA that need a round-wrap row
   int32_t max_long = 0;
+  // Warps per pair GS and pairs per item P (P * GS <= W) per query, two plans:
+  //  latency-first: GS = min(strips, W) (fewest rounds per pair), P = W / GS;
+  //  efficiency-first: the fewest idle warp-rounds -- ns strips over GS warps take
+  //    ceil(ns / GS) rounds and W - P * GS warps idle -- ties to the larger GS, at
+  //    most max(ceil(ns / W), 5) rounds.
+  // The plan with the smaller modelled makespan max(longest item, CTA-steps / CTA
+  // slots) wins: few long pairs (C3's tall-query tail) want short items, a long-only
+  // database (C4) wants busy warps.  The combined single-query launch keeps one
+  // pair per item.
+  std::vector<int> gs_lat(order.size(), 1), gs_eff(order.size(), 1);
+  double span_lat = 0, span_eff = 0, work_lat = 0, work_eff = 0;
+  for (size_t k = 0; k < order.size(); ++k) {
+    const int nl = qnlong[k];
+    if (nl <= 0) continue;
+    const int ns = gl[k].n_strips;
+    int ge = std::min(ns, W);
+    double best_eff = -1;
+    for (int g = std::min(ns, W); g >= 1; --g) {
+      const int p = W / g, rr = (ns + g - 1) / g;
+      if (rr > std::max((ns + W - 1) / W, 5)) continue;  // bounds the item's critical path
+      const double eff = double(p) * ns / (double(W) * rr);
+      if (eff > best_eff + 1e-9) { best_eff = eff; ge = g; }
+    }
+    gs_lat[k] = std::min(ns, W);
+    gs_eff[k] = ge;
+    for (int pl = 0; pl < 2; ++pl) {
+      const int g = pl == 0 ? gs_lat[k] : gs_eff[k], P = W / g;
+      const double rounds = double((ns + g - 1) / g), fill = double(g - 1) * (LINK_LAG_STEPS + 64);
+      double& span = pl == 0 ? span_lat : span_eff;
+      double& work = pl == 0 ? work_lat : work_eff;
+      span = std::max(span, rounds * double(db->pairs[0].len + 64) + fill);
+      for (int it = 0; it * P < nl; ++it) work += rounds * double(db->pairs[size_t(it * P)].len + 64) + fill;
+    }
+  }
+  const double long_slots = double(h->sms) * ((any_q2 || any_m0) ? 1.0 : 2.0);  // SM-exclusive when forked
+  const bool plan_eff = !combined && std::max(span_eff, work_eff / long_slots) <
+                                         std::max(span_lat, work_lat / long_slots);
   for (size_t k = 0; k < order.size(); ++k) {
     const int nl = qnlong[k];
     if (nl <= 0) continue;
@@ -803,22 +841,8 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
     d.n_strips = gl[k].n_strips;
     d.qidx = order[k];
     d.n_long = nl;
-    // warps per pair GS and pairs per item P (P * GS <= W): the fewest idle warp-rounds
-    // (ns strips over GS warps take ceil(ns / GS) rounds; W - P * GS warps idle), ties to
-    // the larger GS (fewer rounds: a shorter critical path per item); at most
-    // max(ceil(ns / W), 5) rounds.  The combined
-    // single-query launch keeps one pair per item.
     const int ns = gl[k].n_strips;
-    int GS = std::min(ns, W), P = combined ? 1 : W / GS;
-    if (!combined) {
-      double best_eff = -1;
-      for (int g = std::min(ns, W); g >= 1; --g) {
-        const int p = W / g, rr = (ns + g - 1) / g;
-        if (rr > std::max((ns + W - 1) / W, 5)) continue;  // bounds the item's critical path
-        const double eff = double(p) * ns / (double(W) * rr);
-        if (eff > best_eff + 1e-9) { best_eff = eff; GS = g; P = p; }
-      }
-    }
+    const int GS = plan_eff ? gs_eff[k] : gs_lat[k], P = combined ? 1 : W / GS;
     d.pack = P;
     d.gs = GS;
     if (ns > GS) wrap_groups = std::max(wrap_groups, P);
@@ -991,7 +1015,10 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
   }
   if (long_items > 0 && !combined) {
     int smem = smem_long;
-    if (fork) smem = std::max(smem, 200 * 1024);  // SM-exclusive (see above)
+    // SM-exclusive when forked (see above); measured on C3 against co-resident long CTAs
+    // (1 per SM), grids capped at 16 / 32 CTAs and a serial long-then-short order:
+    // 1,142 vs 1,163 / 1,204 / 1,157 / 1,154 ms (profiles/r02_ab_long_placement.txt)
+    if (fork) smem = std::max(smem, 200 * 1024);
     const int occ = long_max_ctas_per_sm(smem, nib);
     if (occ <= 0) fail(SW_ECUDA, "long-pair kernel does not fit on an SM");
     const int grid = int(std::max<int64_t>(1, std::min<int64_t>(long_items, int64_t(occ) * h->sms)));

@@ -12,9 +12,11 @@ sys.path.insert(0, os.path.dirname(os.path.dirname(os.path.abspath(__file__))))
 import swgen  # noqa: E402
 import paper_conf_icpp_kedad_sidhoummmmt14_b200 as sw  # noqa: E402
 
-cases = [(35000, 2, 35213), (35000, 600, 35213), (5000, 2, 35213), (35000, 2, 4000), (20000, 600, 7000)]
+cases = [(35000, 2, 35213), (35000, 600, 35213), (5000, 2, 35213), (35000, 2, 4000), (20000, 600, 7000),
+         (4096, 2, 35213), (512, 2, 35213), (512, 592, 35213), (1024, 2, 35213), (8192, 2, 35213)]
 rng = np.random.default_rng(1)
 h = sw.Handle(0, timing=True)
+h.set_option("t_long", 64)
 for M, K, L in cases:
     dc, do = swgen.random_seqs(rng, K, L, L)
     qc, qo = swgen.random_seqs(rng, 1, M, M)
@@ -29,6 +31,9 @@ for M, K, L in cases:
     torch.cuda.synchronize()
     ms = e0.elapsed_time(e1)
     cells = float(M) * K * L
-    print(json.dumps({"M": M, "K": K, "L": L, "ms": round(ms, 2), "GCUPS": round(cells / ms / 1e6, 1),
+    strips = (M + 511) // 512
+    print(json.dumps({"M": M, "K": K, "L": L, "strips": strips, "ms": round(ms, 3),
+                      "ns_per_step_if_8_warps": round(ms * 1e6 / (((strips + 7) // 8) * (L + 64) + min(strips, 8) * 96), 1),
+                      "GCUPS": round(cells / ms / 1e6, 1),
                       "per_item_GCUPS": round(cells / min(K // 2 or 1, 296) / ms / 1e6, 2)}), flush=True)
     db.free()

@@ -741,6 +741,15 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
     for (int k : sl.A) qnlong[size_t(k)] = sl.nlong;
     for (int k : sl.B) qnlong[size_t(k)] = sl.nlong;
   }
+  // single-query searches with long pairs run as ONE combined launch (long items
+  // first, one pair per item); otherwise the long kernel packs short queries' pairs
+  bool any_q2 = false, any_m0 = false, any_long = false;
+  for (auto& sl : slots) {
+    if (sl.nlong < np) (sl.mode == 1 ? any_q2 : any_m0) = true;
+    if (sl.nlong > 0) any_long = true;
+  }
+  const bool combined = any_long && any_m0 && !any_q2;
+  const int LR = combined ? LONG_R_COMBINED : LONG_R;  // rows per lane of the long path
   // ---- profiles: long geometry per query (if it has long pairs); short geometry per slot
   const int LB2 = (((R1 / 4) | 1) * 16);
   // Query-pair profile rows are LDS.128 per lane: a quarter-warp phase holds two
@@ -757,7 +766,7 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
   std::vector<ProfGeom> gl;
   std::vector<size_t> off_l;
   for (size_t k = 0; k < order.size(); ++k) {
-    gl.push_back(make_geom(32, LONG_R, ms[k], alpha, /*long_mode=*/true));
+    gl.push_back(make_geom(32, LR, ms[k], alpha, /*long_mode=*/true));
     off_l.push_back(total);
     total += qnlong[k] > 0 ? size_t(gl.back().n_strips) * gl.back().SB : 0;
   }
@@ -774,14 +783,6 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
     return double(db->len_prefix[size_t(p1)] - db->len_prefix[size_t(p0)]);
   };
   auto pair_res_sum = [&](int p0, int p1) { return db->res_prefix[size_t(p1)] - db->res_prefix[size_t(p0)]; };
-  // single-query searches with long pairs run as ONE combined launch (long items
-  // first, one pair per item); otherwise the long kernel packs short queries' pairs
-  bool any_q2 = false, any_m0 = false, any_long = false;
-  for (auto& sl : slots) {
-    if (sl.nlong < np) (sl.mode == 1 ? any_q2 : any_m0) = true;
-    if (sl.nlong > 0) any_long = true;
-  }
-  const bool combined = any_long && any_m0 && !any_q2;
   if (small_ctas && !combined) {  // (a combined launch needs whole CTAs for its long items)
     NT0 = 32;
     NG0 = NT0 / G0;
@@ -827,7 +828,7 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
       for (int it = 0; it * P < nl; ++it) work += rounds * double(db->pairs[size_t(it * P)].len + 64) + fill;
     }
   }
-  const double long_slots = double(h->sms) * ((any_q2 || any_m0) ? 1.0 : 2.0);  // SM-exclusive when forked
+  const double long_slots = double(h->sms);  // the long kernel holds one CTA per SM (LONG_R = 32)
   const bool plan_eff = !combined && std::max(span_eff, work_eff / long_slots) <
                                          std::max(span_lat, work_lat / long_slots);
   for (size_t k = 0; k < order.size(); ++k) {
@@ -853,7 +854,7 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
     ldesc.push_back(d);
     long_items += (nl + d.pack - 1) / d.pack;
     max_long = std::max(max_long, db->pairs[0].len);
-    out.cells_computed += 2.0 * (pair_len_sum(0, nl) + 64.0 * nl) * double(gl[k].n_strips) * 32 * LONG_R;
+    out.cells_computed += 2.0 * (pair_len_sum(0, nl) + 64.0 * nl) * double(gl[k].n_strips) * 32 * LR;
   }
   // ---- short work: slots per mode
   std::vector<SlotDesc> sdesc(slots.size());

@@ -538,13 +538,13 @@ struct LongShared {
   uint32_t best[LONG_W];
 };
 
-template <bool NIB>
+template <bool NIB, int LR>
 __device__ __forceinline__ void long_item(const LongArgs& a, int item, uint8_t* smem, LongShared& sh) {
   constexpr int W = LONG_W;
   // A producer may run LONG_RING - 4 steps ahead of its consumer's last published
   // consumption; the consumer starts only once the producer is ioff + 4 +
   // LINK_LAG steps in, so the ring must hold more than that (else both wait).
-  static_assert(LONG_RING - 4 >= (32 * SubLanes<LONG_R>::V - 1) + 4 + LINK_LAG + 16, "ring too short for the lag");
+  static_assert(LONG_RING - 4 >= (32 * SubLanes<LR>::V - 1) + 4 + LINK_LAG + 16, "ring too short for the lag");
   uint2* rings = reinterpret_cast<uint2*>(smem);                       // [W - 1][LONG_RING]
   uint8_t* lprof = smem + (W - 1) * LONG_RING * sizeof(uint2);         // [W][SBL]
   int* s_prog = sh.prog;
@@ -569,7 +569,7 @@ __device__ __forceinline__ void long_item(const LongArgs& a, int item, uint8_t* 
     PairRec pr;
     if (active) pr = a.pairs[pidx];
     else { pr.off = 0; pr.len = 0; pr.id0 = -1; pr.id1 = -1; }
-    constexpr int VG = 32 * SubLanes<LONG_R>::V;
+    constexpr int VG = 32 * SubLanes<LR>::V;
     const int T = pr.len + VG;
     uint32_t best = 0;
     uint8_t* myprof = lprof + warp * a.SBL;
@@ -609,7 +609,7 @@ __device__ __forceinline__ void long_item(const LongArgs& a, int item, uint8_t* 
       ch.out_prog = &s_prog[cbase + j];
       const void* pstream = NIB ? static_cast<const void*>(reinterpret_cast<const uint8_t*>(a.stream) + pr.off)
                                 : static_cast<const void*>(a.stream + pr.off);
-      strip_pass<32, LONG_R, true, false, LONG_US, NIB>(myprof, a.LSL, a.LBL, pstream, pr.len, T, lane, rd, wr,
+      strip_pass<32, LR, true, false, LONG_US, NIB>(myprof, a.LSL, a.LBL, pstream, pr.len, T, lane, rd, wr,
                                                    nullptr, nullptr, ch, a.code_pad2, a.nGe, a.nGsGe, best);
     }
 #pragma unroll
@@ -663,7 +663,7 @@ __global__ void __launch_bounds__(NT, 2) short_kernel(ShortArgs as) {
 // the short path's register allocation apart from it.
 template <bool NIB>
 __device__ __noinline__ void long_item_call(const LongArgs& a, int item, uint8_t* smem, LongShared& sh) {
-  long_item<NIB>(a, item, smem, sh);
+  long_item<NIB, LONG_R_COMBINED>(a, item, smem, sh);
 }
 
 // Single-query searches with long pairs (C1/C2): ONE persistent launch, the long
@@ -698,7 +698,7 @@ __global__ void __launch_bounds__(NT, 2) combined_m0_kernel(ShortArgs as, LongAr
 // for a short-pair CTA), so the co-resident short warps do not stretch the
 // critical path of the longest pairs.
 template <bool NIB>
-__global__ void __launch_bounds__(LONG_W * 32, 2) long_kernel(LongArgs al) {
+__global__ void __launch_bounds__(LONG_W * 32, 1) long_kernel(LongArgs al) {
   extern __shared__ __align__(128) uint8_t smem[];
   __shared__ int s_item;
   __shared__ LongShared sh;
@@ -708,7 +708,7 @@ __global__ void __launch_bounds__(LONG_W * 32, 2) long_kernel(LongArgs al) {
     const int item = s_item;
     __syncthreads();
     if (item >= al.n_items) break;
-    long_item<NIB>(al, item, smem, sh);
+    long_item<NIB, LONG_R>(al, item, smem, sh);
   }
 }
 
@@ -947,7 +947,11 @@ __global__ void __launch_bounds__(RESCORE_WARPS * 32) rescore_kernel(RescoreArgs
           }
           v = __shfl_sync(FULL, v, 0);
           if (v >= need) { seen = v; break; }
-          __nanosleep(in_gpu ? 256 : 64);
+#ifndef SW_RS_SLEEP_GPU
+#define SW_RS_SLEEP_GPU 256
+#define SW_RS_SLEEP_CTA 64
+#endif
+          __nanosleep(in_gpu ? SW_RS_SLEEP_GPU : SW_RS_SLEEP_CTA);
         }
         if (in_gpu) __threadfence();
       };

@@ -58,7 +58,12 @@ struct ProfGeom {
 // Rows per lane of the intra-task (long pair) geometry, G = 32 lanes; profile
 // unit-interleaved ([letter][unit][lane][8 B]): dense and bank-conflict-free (the
 // 16 lanes of an LDS.64 phase hit 16 distinct 8-byte slots whatever letters they read)
-constexpr int LONG_R = 16;
+// Rows per lane of the long kernel (32: one CTA of 8 warps per SM, 25.6 KB of int8
+// profile per warp; the per-step ring I/O, waits and code handling amortised over 32
+// rows) and of the long path inside the combined single-query kernel (16: it shares
+// the SM with a second CTA of short items).
+constexpr int LONG_R = 32;
+constexpr int LONG_R_COMBINED = 16;
 constexpr int LONG_US = 32 * 8;     // bytes between a lane's consecutive 8-byte units in the long profile
 constexpr int LONG_RING = 128;      // steps held by a shared-memory link ring between two warps of a CTA
 

@@ -527,14 +527,14 @@ def test_small_search_one_group_ctas(small):
 
 def test_long_only_search_tall_queries():
     """A search whose pairs are all long (every DB sequence longer than t_long)
-    runs the long kernel alone: tall queries (26 and 69 strips) chain their
-    strips over the warps of one CTA in rounds (the round wrap through global
-    memory); queries of fewer strips than the CTA's warps pack several pairs per
-    item.  Equals the oracle."""
+    runs the long kernel alone: tall queries chain their strips over the warps
+    of one CTA in rounds (the round wrap through global memory); the host packs
+    several pairs per item when that leaves fewer warps idle.  Equals the oracle."""
     rng = np.random.default_rng(240)
     dc, do = _seqs(list(rng.integers(70, 900, size=24)) + [3001, 1500], rng)
-    # 26 / 69 strips: 8 warps per pair; 4 strips: 2 pairs of 4 warps; 10 strips: 4 pairs of
-    # 2 warps (5 rounds, one round-wrap row per pair group); 20 strips: 2 pairs of 4 warps
+    # 1,024-row strips (32 lanes x 32 rows): 13 / 35 strips over 8 warps per pair (2 / 5
+    # rounds, the round wrap through global memory); 2 strips: 4 pairs of 2 warps; 5 and
+    # 10 strips: 8 pairs of 1 warp / 4 pairs of 2 warps (one round-wrap row per pair group)
     for ql in ([13000, 100, 700], [35000, 2000], [5000, 10000, 300]):
         qc, qo = _seqs(ql, rng)
         got = gpu_scores(qc, qo, dc, do, opts={"t_long": 64})

@@ -1076,7 +1076,7 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
     if (with_long) smem = std::max(smem, smem_long);  // an item is short or long: the two uses share smem
     const bool cg = c.nGe == 0xfffefffeu && c.nGsGe == 0xfff4fff4u && h->opt_const_gaps != 0;
     const int nt = mode == 1 ? NT1 : NT0;
-    const int occ = with_long ? combined_max_ctas_per_sm(G, R, smem, nib)
+    const int occ = with_long ? combined_max_ctas_per_sm(G, R, smem, nib, cg)
                               : short_max_ctas_per_sm(mode, G, R, smem, cg, nib, nt);
     if (occ <= 0) fail(SW_ECUDA, "short-pair kernel does not fit on an SM");
     const int64_t items = int64_t(n_short) + (with_long ? long_items : 0);
@@ -1107,7 +1107,7 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
       al.wrap_groups = wrap_groups;
       SW_CK(h->wrap.ensure(size_t(grid) * wrap_groups * al.wcap * sizeof(uint2)));
       al.wrap = h->wrap.as<uint2>();
-      SW_CK(launch_combined(G, R, grid, smem, as, al, c.st, nib));
+      SW_CK(launch_combined(G, R, grid, smem, as, al, c.st, nib, cg));
     } else {
       SW_CK(launch_short(mode, G, R, grid, smem, as, c.st, cg, nib, nt));
     }

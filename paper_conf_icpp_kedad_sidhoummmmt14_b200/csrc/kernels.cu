@@ -669,7 +669,7 @@ __device__ __noinline__ void long_item_call(const LongArgs& a, int item, uint8_t
 // Single-query searches with long pairs (C1/C2): ONE persistent launch, the long
 // items first (costliest), then the short items, so the longest pairs start at
 // once and the SMs that finish them move on to short items.
-template <int G, int R, int NT, bool NIB = false>
+template <int G, int R, int NT, bool NIB = false, bool CG = false>
 __global__ void __launch_bounds__(NT, 2) combined_m0_kernel(ShortArgs as, LongArgs al) {
   extern __shared__ __align__(128) uint8_t smem[];
   __shared__ int s_item;
@@ -687,7 +687,7 @@ __global__ void __launch_bounds__(NT, 2) combined_m0_kernel(ShortArgs as, LongAr
       long_item_call<NIB>(al, item, smem, sh);
       loaded = -1;  // the long item overwrote the strip profile
     } else {
-      short_item<G, R, NT, false, false, NIB>(as, item - al.n_items, smem, loaded, ps);
+      short_item<G, R, NT, false, CG, NIB>(as, item - al.n_items, smem, loaded, ps);
     }
   }
 }
@@ -807,7 +807,12 @@ cudaError_t launch_short(int mode, int G, int R, int grid, int smem_bytes, const
 }
 
 typedef void (*combined_fn)(ShortArgs, LongArgs);
-static combined_fn pick_combined(int G, int R, bool nib) {
+static combined_fn pick_combined(int G, int R, bool nib, bool cg) {
+  if (cg && !nib) {
+#define X(g, r) if (G == g && R == r) return combined_m0_kernel<g, r, SCORE_NT, false, true>;
+    SW_CG_CASES(X)
+#undef X
+  }
   if (nib) {
 #define X(g, r) if (G == g && R == r) return combined_m0_kernel<g, r, SCORE_NT, true>;
     SW_NIB_CASES(X)
@@ -820,14 +825,14 @@ static combined_fn pick_combined(int G, int R, bool nib) {
   return nullptr;
 }
 
-int combined_max_ctas_per_sm(int G, int R, int smem_bytes, bool nib) {
-  combined_fn f = pick_combined(G, R, nib);
+int combined_max_ctas_per_sm(int G, int R, int smem_bytes, bool nib, bool cg) {
+  combined_fn f = pick_combined(G, R, nib, cg);
   return f ? occupancy(reinterpret_cast<const void*>(f), SCORE_NT, smem_bytes) : 0;
 }
 
 cudaError_t launch_combined(int G, int R, int grid, int smem_bytes, const ShortArgs& as, const LongArgs& al,
-                            cudaStream_t st, bool nib) {
-  combined_fn f = pick_combined(G, R, nib);
+                            cudaStream_t st, bool nib, bool cg) {
+  combined_fn f = pick_combined(G, R, nib, cg);
   if (!f) return cudaErrorInvalidValue;
   if (smem_bytes > 48 * 1024) {
     cudaError_t e = cudaFuncSetAttribute(f, cudaFuncAttributeMaxDynamicSharedMemorySize, smem_bytes);

@@ -209,9 +209,9 @@ cudaError_t launch_short(int mode, int G, int R, int grid, int smem_bytes, const
 int long_max_ctas_per_sm(int smem_bytes, bool nib = false);
 cudaError_t launch_long(int grid, int smem_bytes, const LongArgs& a, cudaStream_t st, bool nib = false);
 // single-query searches with long pairs: long items and mode-0 short items in one launch
-int combined_max_ctas_per_sm(int G, int R, int smem_bytes, bool nib = false);
+int combined_max_ctas_per_sm(int G, int R, int smem_bytes, bool nib = false, bool cg = false);
 cudaError_t launch_combined(int G, int R, int grid, int smem_bytes, const ShortArgs& as, const LongArgs& al,
-                            cudaStream_t st, bool nib = false);
+                            cudaStream_t st, bool nib = false, bool cg = false);
 cudaError_t launch_rescore(int grid, const RescoreArgs& a, cudaStream_t st);
 // scores[q * stride + cols[c]] = 0 for every query q < nq and column c < ncols
 cudaError_t launch_zero_columns(int32_t* scores, int64_t stride, int nq, const int64_t* cols, int64_t ncols,

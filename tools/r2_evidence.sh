@@ -1,7 +1,7 @@
 #!/bin/bash
-# Round-2 end-of-round evidence in one call: GPU suite + smoke, bench lines (C3 default with the
-# cpu_baseline, C4, C2, C1, Table V), the oracle arm, the C3 launch list, ncu --set full of the
-# dominant kernels (C3 slice, C4, C2), C5 on one GPU and through the 2-rank path.
+# Round-2 end-of-round evidence, part 1: bench lines (C3 default with the cpu_baseline, C4, C2,
+# C1, Table V), the oracle arm, the C3 launch list, smoke, the GPU suite (part 2:
+# tools/r2_evidence_ncu.sh).
 T=${1:-r2z}; mkdir -p gpurun_out
 nvidia-smi --query-gpu=name,clocks.sm,clocks.max.sm,power.draw --format=csv > gpurun_out/${T}_smi.txt
 timeout 900 python bench.py > gpurun_out/${T}_bench_c3.json 2> gpurun_out/${T}_bench_c3.err
@@ -11,14 +11,6 @@ done
 timeout 900 python bench.py --impl reference --steps 2 --warmup 3 > gpurun_out/${T}_bench_ref.json 2> gpurun_out/${T}_bench_ref.err
 timeout 900 ncu --metrics gpu__time_duration.sum --clock-control none --csv --log-file gpurun_out/${T}_launches_c3.csv \
   python bench.py --steps 1 --warmup 1 --no-cpu-baseline --e2e-steps 0 > gpurun_out/${T}_launches_c3.log 2>&1
-PROF_WORKLOAD=c3 PROF_NDB=100000 PROF_REPS=1 timeout 900 ncu --set full --clock-control none --import-source on \
-  -k regex:short_kernel -c 1 -o gpurun_out/${T}_full_c3sub -f python tools/prof_one.py > gpurun_out/${T}_full_c3sub.log 2>&1
-PROF_WORKLOAD=c4 PROF_REPS=1 timeout 900 ncu --set full --clock-control none --import-source on \
-  -k regex:long_kernel -c 1 -o gpurun_out/${T}_full_c4 -f python tools/prof_one.py > gpurun_out/${T}_full_c4.log 2>&1
-PROF_WORKLOAD=c2 PROF_REPS=1 timeout 900 ncu --set full --clock-control none --import-source on \
-  -k regex:combined -c 1 -o gpurun_out/${T}_full_c2 -f python tools/prof_one.py > gpurun_out/${T}_full_c2.log 2>&1
 timeout 300 python -c "import __graft_entry__ as g; g.smoke()" > gpurun_out/${T}_smoke.txt 2>&1
 timeout 3000 python -m pytest tests -q -m gpu -rf --timeout=1200 > gpurun_out/${T}_gpu_tests.txt 2>&1
-timeout 1800 python bench.py --workload c5 --steps 1 --warmup 1 --e2e-steps 0 --no-cpu-baseline > gpurun_out/${T}_bench_c5.json 2> gpurun_out/${T}_bench_c5.err
-bash tools/c5_multirank.sh ${T}
 echo done

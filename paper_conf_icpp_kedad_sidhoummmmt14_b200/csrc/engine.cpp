@@ -748,7 +748,10 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
     if (sl.nlong < np) (sl.mode == 1 ? any_q2 : any_m0) = true;
     if (sl.nlong > 0) any_long = true;
   }
-  const bool combined = any_long && any_m0 && !any_q2;
+#ifndef SW_NO_COMBINED
+#define SW_NO_COMBINED 0
+#endif
+  const bool combined = any_long && any_m0 && !any_q2 && !SW_NO_COMBINED;
   const int LR = combined ? LONG_R_COMBINED : LONG_R;  // rows per lane of the long path
   // ---- profiles: long geometry per query (if it has long pairs); short geometry per slot
   const int LB2 = (((R1 / 4) | 1) * 16);

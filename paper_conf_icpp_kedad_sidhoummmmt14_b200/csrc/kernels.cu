@@ -662,7 +662,12 @@ __global__ void __launch_bounds__(NT, 2) short_kernel(ShortArgs as) {
 // A long item as an out-of-line call: the combined single-query kernel below keeps
 // the short path's register allocation apart from it.
 template <bool NIB>
-__device__ __noinline__ void long_item_call(const LongArgs& a, int item, uint8_t* smem, LongShared& sh) {
+#ifdef SW_COMB_INLINE
+__device__ __forceinline__
+#else
+__device__ __noinline__
+#endif
+void long_item_call(const LongArgs& a, int item, uint8_t* smem, LongShared& sh) {
   long_item<NIB, LONG_R_COMBINED>(a, item, smem, sh);
 }
 

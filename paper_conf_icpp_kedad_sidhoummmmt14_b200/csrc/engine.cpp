@@ -748,10 +748,8 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
     if (sl.nlong < np) (sl.mode == 1 ? any_q2 : any_m0) = true;
     if (sl.nlong > 0) any_long = true;
   }
-#ifndef SW_NO_COMBINED
-#define SW_NO_COMBINED 0
-#endif
-  const bool combined = any_long && any_m0 && !any_q2 && !SW_NO_COMBINED;
+  const bool combined = any_long && any_m0 && !any_q2;  // (vs the forked long kernel on C2: 20.7 vs 28.7 ms,
+                                                        //  profiles/r02_ab_combined_forms.txt)
   const int LR = combined ? LONG_R_COMBINED : LONG_R;  // rows per lane of the long path
   // ---- profiles: long geometry per query (if it has long pairs); short geometry per slot
   const int LB2 = (((R1 / 4) | 1) * 16);
@@ -824,11 +822,11 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
     gs_eff[k] = ge;
     for (int pl = 0; pl < 2; ++pl) {
       const int g = pl == 0 ? gs_lat[k] : gs_eff[k], P = W / g;
-      const double rounds = double((ns + g - 1) / g), fill = double(g - 1) * (LINK_LAG_STEPS + 64);
+      const double rounds = double((ns + g - 1) / g), fill = double(g - 1) * (LINK_LAG_STEPS + 32 * LONG_V);
       double& span = pl == 0 ? span_lat : span_eff;
       double& work = pl == 0 ? work_lat : work_eff;
-      span = std::max(span, rounds * double(db->pairs[0].len + 64) + fill);
-      for (int it = 0; it * P < nl; ++it) work += rounds * double(db->pairs[size_t(it * P)].len + 64) + fill;
+      span = std::max(span, rounds * double(db->pairs[0].len + 32 * LONG_V) + fill);
+      for (int it = 0; it * P < nl; ++it) work += rounds * double(db->pairs[size_t(it * P)].len + 32 * LONG_V) + fill;
     }
   }
   const double long_slots = double(h->sms);  // the long kernel holds one CTA per SM (LONG_R = 32)
@@ -1004,7 +1002,7 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
     al.n_items = int(long_items);
     al.lmap = h->lmap.as<int2>();
     al.SBL = l0.SB; al.LSL = l0.LS; al.LBL = l0.LB;
-    smem_long = (W - 1) * LONG_RING * int(sizeof(uint2)) + W * l0.SB;
+    smem_long = (W - 1) * (combined ? LONG_RING : LONG_RING_K) * int(sizeof(uint2)) + W * l0.SB;
     al.wcap = max_long + 64 + 8;
     al.stream = db->stream.as<uint16_t>();
     al.pairs = db->dpairs.as<PairRec>();

@@ -822,11 +822,11 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
     gs_eff[k] = ge;
     for (int pl = 0; pl < 2; ++pl) {
       const int g = pl == 0 ? gs_lat[k] : gs_eff[k], P = W / g;
-      const double rounds = double((ns + g - 1) / g), fill = double(g - 1) * (LINK_LAG_STEPS + 32 * LONG_V);
+      const double rounds = double((ns + g - 1) / g), fill = double(g - 1) * (LINK_LAG_STEPS + 64);
       double& span = pl == 0 ? span_lat : span_eff;
       double& work = pl == 0 ? work_lat : work_eff;
-      span = std::max(span, rounds * double(db->pairs[0].len + 32 * LONG_V) + fill);
-      for (int it = 0; it * P < nl; ++it) work += rounds * double(db->pairs[size_t(it * P)].len + 32 * LONG_V) + fill;
+      span = std::max(span, rounds * double(db->pairs[0].len + 64) + fill);
+      for (int it = 0; it * P < nl; ++it) work += rounds * double(db->pairs[size_t(it * P)].len + 64) + fill;
     }
   }
   const double long_slots = double(h->sms);  // the long kernel holds one CTA per SM (LONG_R = 32)
@@ -1002,7 +1002,7 @@ static void launch_all(LaunchCtx& c, const std::vector<int64_t>& qlen, const std
     al.n_items = int(long_items);
     al.lmap = h->lmap.as<int2>();
     al.SBL = l0.SB; al.LSL = l0.LS; al.LBL = l0.LB;
-    smem_long = (W - 1) * (combined ? LONG_RING : LONG_RING_K) * int(sizeof(uint2)) + W * l0.SB;
+    smem_long = (W - 1) * LONG_RING * int(sizeof(uint2)) + W * l0.SB;
     al.wcap = max_long + 64 + 8;
     al.stream = db->stream.as<uint16_t>();
     al.pairs = db->dpairs.as<PairRec>();

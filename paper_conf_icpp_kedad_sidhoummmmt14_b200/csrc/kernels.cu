@@ -188,20 +188,12 @@ __device__ __forceinline__ void wait_geq(const int* p, int need, int& seen, int 
 // NIB: the pair's columns are bytes of two 4-bit codes (nucleotide DBs, SURVEY 8(f)
 // f4): lane 0 loads 4 columns per 32-bit word and spreads each byte into the
 // 16-bit pair word (two 8-bit codes) the rest of the pass uses.
-// VV: sub-lanes per lane (0: SubLanes<R>::V; 4: four skewed chains of R/4 rows, single-query
-// form only -- the long kernel, whose 2 warps per scheduler need the extra independent
-// chains).  RING: steps held by a link ring (the lag grows with the wave width).
-template <int V>
-struct LinkRing { static constexpr int N = V == 4 ? 256 : 128; };
-template <int G, int R, bool LINKED, bool Q2 = false, int US = (Q2 ? 16 : ((R % 8 == 0) ? 8 : 4)), bool NIB = false,
-          int VV = 0>
+template <int G, int R, bool LINKED, bool Q2 = false, int US = (Q2 ? 16 : ((R % 8 == 0) ? 8 : 4)), bool NIB = false>
 __device__ __forceinline__ void strip_pass(const uint8_t* sprof, int LS, int LB, const void* pstream, int L,
                                            int T, int k, bool rd, bool wr, const uint2* __restrict__ rp,
                                            uint2* __restrict__ wp, const Chain& ch, uint32_t code_pad2,
                                            uint32_t nGe, uint32_t nGsGe, uint32_t& best, uint32_t shift = 0) {
-  constexpr int V = VV ? VV : SubLanes<R>::V;
-  static_assert(V != 4 || (!Q2 && R % 32 == 0), "four sub-lanes: single-query form, 8-row units");
-  constexpr int LONG_RING = LinkRing<V>::N;
+  constexpr int V = SubLanes<R>::V;
   constexpr int VG = V * G;   // width of the wave in sub-lanes
   constexpr int RH = R / V;   // rows per sub-lane
   // code-ahead pipeline (below): single-query short items only -- measured C2 +3 %; the
@@ -223,10 +215,6 @@ __device__ __forceinline__ void strip_pass(const uint8_t* sprof, int LS, int LB,
   uint32_t hdiag1 = 0, cH = 0, cF = 0, pC = code_pad2;
   const uint32_t pad_row = sbase + (code_pad2 & 0xffu) * LS + laneoff;
   uint32_t ppa = pad_row, ppb = pad_row;
-  // V = 4: sub-lanes 2 and 3 (column t-2, t-3): inputs = sub-lane 1 / 2 outputs of the
-  // previous step, profile rows of sub-lane 0's letter two / three steps ago
-  uint32_t hdiag2 = 0, hdiag3 = 0, cH1 = 0, cF1 = 0, cH2 = 0, cF2 = 0, pC2 = code_pad2, pC3 = code_pad2;
-  uint32_t ppa2 = pad_row, ppb2 = pad_row, ppa3 = pad_row, ppb3 = pad_row;
   // input index of sub-lane 0 of lane 0 for column c: c + VG - 1 (producer step)
   const int ioff = VG - 1;
   int seen_in = -1, seen_out = -1;
@@ -323,7 +311,7 @@ __device__ __forceinline__ void strip_pass(const uint8_t* sprof, int LS, int LB,
       uint32_t rC;
       if (CA) {
         rC = nC;
-        uint32_t xC = __shfl_up_sync(FULL, V == 4 ? pC3 : V == 2 ? pC : rC, 1, G);  // this lane's next code
+        uint32_t xC = __shfl_up_sync(FULL, V == 2 ? pC : rC, 1, G);  // this lane's code of the next step
         if (lead) xC = (j < 3) ? code_at(cwc, j + 1) : code_at(cwnc, 0);
         nC = xC;
       } else {
@@ -343,29 +331,7 @@ __device__ __forceinline__ void strip_pass(const uint8_t* sprof, int LS, int LB,
         pa = sbase + (rC & 0xffu) * LS + laneoff;
         pb = sbase + (rC >> 8) * LS + laneoff;
       }
-      if constexpr (V == 4) {
-        // sub-lane u (rows u*RH .. u*RH+RH-1) at column t-u, deepest first: each reads the
-        // outputs its upper sub-lane produced in the previous step before they are replaced
-        uint32_t h3 = cH2, f3 = cF2;
-        gotoh_rows_inplace<R, 3 * RH, 4 * RH, false, US>(HA, E, best, hdiag3, ppa3, ppb3, h3, f3, nGe, nGsGe);
-        uint32_t h2 = cH1, f2 = cF1;
-        gotoh_rows_inplace<R, 2 * RH, 3 * RH, false, US>(HA, E, best, hdiag2, ppa2, ppb2, h2, f2, nGe, nGsGe);
-        uint32_t h1 = cH, f1 = cF;
-        gotoh_rows_inplace<R, RH, 2 * RH, false, US>(HA, E, best, hdiag1, ppa, ppb, h1, f1, nGe, nGsGe);
-        gotoh_rows_inplace<R, 0, RH, false, US>(HA, E, best, hdiag, pa, pb, rH, rF, nGe, nGsGe);
-        cH2 = h2; cF2 = f2;
-        cH1 = h1; cF1 = f1;
-        cH = rH; cF = rF;
-        ppa3 = ppa2; ppb3 = ppb2;
-        ppa2 = ppa; ppb2 = ppb;
-        ppa = pa; ppb = pb;
-        sH = h3;
-        sF = f3;
-        sC = pC3;  // the code of sub-lane 3 (sub-lane 0's, three steps ago): the next lane's next code
-        pC3 = pC2;
-        pC2 = pC;
-        pC = rC;
-      } else if constexpr (V == 2) {
+      if constexpr (V == 2) {
         uint32_t h1 = cH, f1 = cF;
         if constexpr (Q2) {  // measured: +3% for the query-pair mode, -2% with the PRMT (mode 0)
           gotoh_rows_dual<R, Q2, US>(HA, E, best, hdiag, pa, pb, rH, rF, hdiag1, ppa, ppb, h1, f1, nGe, nGsGe);
@@ -575,12 +541,10 @@ struct LongShared {
 template <bool NIB, int LR>
 __device__ __forceinline__ void long_item(const LongArgs& a, int item, uint8_t* smem, LongShared& sh) {
   constexpr int W = LONG_W;
-  constexpr int LV = LR == LONG_R ? LONG_V : SubLanes<LR>::V;  // sub-lanes per lane
-  constexpr int LONG_RING = LinkRing<LV>::N;
   // A producer may run LONG_RING - 4 steps ahead of its consumer's last published
   // consumption; the consumer starts only once the producer is ioff + 4 +
   // LINK_LAG steps in, so the ring must hold more than that (else both wait).
-  static_assert(LONG_RING - 4 >= (32 * LV - 1) + 4 + LINK_LAG + 16, "ring too short for the lag");
+  static_assert(LONG_RING - 4 >= (32 * SubLanes<LR>::V - 1) + 4 + LINK_LAG + 16, "ring too short for the lag");
   uint2* rings = reinterpret_cast<uint2*>(smem);                       // [W - 1][LONG_RING]
   uint8_t* lprof = smem + (W - 1) * LONG_RING * sizeof(uint2);         // [W][SBL]
   int* s_prog = sh.prog;
@@ -605,7 +569,7 @@ __device__ __forceinline__ void long_item(const LongArgs& a, int item, uint8_t* 
     PairRec pr;
     if (active) pr = a.pairs[pidx];
     else { pr.off = 0; pr.len = 0; pr.id0 = -1; pr.id1 = -1; }
-    constexpr int VG = 32 * LV;
+    constexpr int VG = 32 * SubLanes<LR>::V;
     const int T = pr.len + VG;
     uint32_t best = 0;
     uint8_t* myprof = lprof + warp * a.SBL;
@@ -645,7 +609,7 @@ __device__ __forceinline__ void long_item(const LongArgs& a, int item, uint8_t* 
       ch.out_prog = &s_prog[cbase + j];
       const void* pstream = NIB ? static_cast<const void*>(reinterpret_cast<const uint8_t*>(a.stream) + pr.off)
                                 : static_cast<const void*>(a.stream + pr.off);
-      strip_pass<32, LR, true, false, LONG_US, NIB, LV>(myprof, a.LSL, a.LBL, pstream, pr.len, T, lane, rd, wr,
+      strip_pass<32, LR, true, false, LONG_US, NIB>(myprof, a.LSL, a.LBL, pstream, pr.len, T, lane, rd, wr,
                                                    nullptr, nullptr, ch, a.code_pad2, a.nGe, a.nGsGe, best);
     }
 #pragma unroll

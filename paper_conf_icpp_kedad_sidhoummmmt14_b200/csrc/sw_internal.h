@@ -66,13 +66,6 @@ constexpr int LONG_R = 32;
 constexpr int LONG_R_COMBINED = 16;
 constexpr int LONG_US = 32 * 8;     // bytes between a lane's consecutive 8-byte units in the long profile
 constexpr int LONG_RING = 128;      // steps held by a shared-memory link ring between two warps of a CTA
-// The long kernel's lanes run four skewed sub-lanes of 8 rows (two chains per warp are
-// too few at 2 warps per scheduler): a 128-sub-lane wave, so its rings hold 256 steps.
-#ifndef SW_LONG_V4
-#define SW_LONG_V4 1
-#endif
-constexpr int LONG_V = SW_LONG_V4 ? 4 : 2;
-constexpr int LONG_RING_K = SW_LONG_V4 ? 256 : 128;
 
 // Long (intra-task) work of one query: pairs [0, n_long) of the DB are scored by
 // the chained warps of one CTA each.

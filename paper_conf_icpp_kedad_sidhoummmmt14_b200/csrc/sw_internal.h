@@ -220,7 +220,8 @@ cudaError_t launch_assemble(const int32_t* src, const AsmBlock* blocks, int n_bl
                             int64_t total, const int32_t* rows, const int64_t* cols, int32_t* out, int64_t N,
                             int sms, cudaStream_t st);
 constexpr int RESCORE_WARPS = 8;
-constexpr int RESCORE_R = 8;
+constexpr int RESCORE_R = 8;  // (C4: 4 rows 13.3 ms, 8 rows 14.9 ms, 16 rows 22 ms per search, profiles/r02_ab_rescore_rows.txt;
+                              //  4 would overflow the (strip << 20) counters for queries over 2^18 rows)
 
 
 // Best local alignment of selected pairs (align.cu).  One item =

@@ -246,6 +246,8 @@ int32_t sw_last_stats(sw_handle_t h, sw_stats_t* out);
  *   "bank_skew"           1: single-query profile copies one per lane group of
  *                         a shared-memory phase at searched bank skews
  *                         (conflict-free; default 1), 0: the linear layout
+ *   "rescore_rows"        rows per lane of the int32 re-score: 0 (default) = 4 when every
+ *                         query has fewer than 2^11 strips of 128 rows, else 8; 8 forces 8
  *   "const_gaps"          1 (default): searches with Gs = 10, Ge = 2 use kernel
  *                         instantiations with the penalties as immediates; 0: the
  *                         runtime-penalty kernels (same results)

@@ -189,6 +189,7 @@ struct sw_handle_s {
   int64_t opt_const_gaps = 1;   // gaps 10/2: the constant-gap kernel instantiations
   int64_t opt_nibble = 1;       // alphabets <= 15: 4-bit DB stream
   int64_t opt_small_ctas = 1;   // latency-bound single-query searches: 32-thread CTAs
+  int64_t opt_rescore_rows = 0; // int32 re-score rows per lane: 0 = automatic (4 or 8), 4, 8
   int64_t opt_crit_min = CRIT_MIN_STEPS;                    // long-pair rule (see launch_all)
   int64_t opt_crit_pct = int64_t(CRIT_FRACTION * 100 + 0.5);
   int64_t opt_align_ws_mb = 2048;  // sw_align: traceback-code workspace per batch
@@ -438,6 +439,9 @@ int32_t sw_set_option(sw_handle_t h, const char* key, int64_t value) {
   } else if (k == "crit_pct") {
     if (value < 1) return set_err(h, SW_EINVAL, "crit_pct must be >= 1");
     h->opt_crit_pct = value;
+  } else if (k == "rescore_rows") {
+    if (value != 0 && value != 4 && value != 8) return set_err(h, SW_EINVAL, "rescore_rows must be 0, 4 or 8");
+    h->opt_rescore_rows = value;
   } else if (k == "small_ctas") {
     h->opt_small_ctas = value;
   } else if (k == "nibble") {
@@ -1241,7 +1245,9 @@ int32_t sw_search(sw_handle_t h, const uint8_t* q_codes, const int64_t* q_offset
       const int32_t Lmax = std::max(max_short, max_long);
       int64_t mmax = 1;
       for (auto L : qlen) mmax = std::max(mmax, L);
-      const int rows_per_strip = 32 * RESCORE_R;
+      const bool r4_ok = mmax <= int64_t(2047) * 32 * 4;  // (strip << 20) counters: < 2^11 strips
+      const int rrows = (h->opt_rescore_rows == 8 || !r4_ok) ? RESCORE_R : 4;
+      const int rows_per_strip = 32 * rrows;
       const int nstrips = int((mmax + rows_per_strip - 1) / rows_per_strip);
       // one round of RESCORE_WARPS strips per CTA (every wait targets an earlier item)
       const int K = std::max(1, (nstrips + RESCORE_WARPS - 1) / RESCORE_WARPS);
@@ -1279,7 +1285,7 @@ int32_t sw_search(sw_handle_t h, const uint8_t* q_codes, const int64_t* q_offset
       r.n_seqs = N;
       r.Gs = gap_open;
       r.Ge = gap_extend;
-      SW_CK(launch_rescore(grid, r, st));
+      SW_CK(launch_rescore(grid, r, st, rrows));
       ++launches;
     }
     if (timing) {

@@ -212,7 +212,8 @@ cudaError_t launch_long(int grid, int smem_bytes, const LongArgs& a, cudaStream_
 int combined_max_ctas_per_sm(int G, int R, int smem_bytes, bool nib = false, bool cg = false);
 cudaError_t launch_combined(int G, int R, int grid, int smem_bytes, const ShortArgs& as, const LongArgs& al,
                             cudaStream_t st, bool nib = false, bool cg = false);
-cudaError_t launch_rescore(int grid, const RescoreArgs& a, cudaStream_t st);
+// rows: rows per lane, RESCORE_R or 4 (only when every query has < 2^11 strips of 128 rows)
+cudaError_t launch_rescore(int grid, const RescoreArgs& a, cudaStream_t st, int rows);
 // scores[q * stride + cols[c]] = 0 for every query q < nq and column c < ncols
 cudaError_t launch_zero_columns(int32_t* scores, int64_t stride, int nq, const int64_t* cols, int64_t ncols,
                                 cudaStream_t st);
@@ -220,8 +221,8 @@ cudaError_t launch_assemble(const int32_t* src, const AsmBlock* blocks, int n_bl
                             int64_t total, const int32_t* rows, const int64_t* cols, int32_t* out, int64_t N,
                             int sms, cudaStream_t st);
 constexpr int RESCORE_WARPS = 8;
-constexpr int RESCORE_R = 8;  // (C4: 4 rows 13.3 ms, 8 rows 14.9 ms, 16 rows 22 ms per search, profiles/r02_ab_rescore_rows.txt;
-                              //  4 would overflow the (strip << 20) counters for queries over 2^18 rows)
+constexpr int RESCORE_R = 8;  // rows per lane; 4 for searches whose queries all have < 2^11 strips of
+                              // 128 rows (C4: 13.3 vs 14.9 ms, 16 rows 22 ms, profiles/r02_ab_rescore_rows.txt)
 
 
 // Best local alignment of selected pairs (align.cu).  One item =

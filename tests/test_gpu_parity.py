@@ -104,14 +104,17 @@ def test_asymmetric_matrix_small_alphabet():
     np.testing.assert_array_equal(got, oracle_scores(qc, qo, dc, do, S=S.astype(np.int32), gs=3, ge=1))
 
 
-def test_forced_overflow_rescore():
-    """A tiny threshold sends most pairs through the int32 re-score path."""
+@pytest.mark.parametrize("rows", [0, 8])
+def test_forced_overflow_rescore(rows):
+    """A tiny threshold sends most pairs through the int32 re-score path (4 rows per
+    lane, the automatic choice here, and 8, the choice for queries of >= 2^11 strips)."""
     rng = np.random.default_rng(14)
     dc, do = _seqs(rng.integers(1, 500, size=120), rng)
     qc, qo = _seqs([200, 900], rng)
     sw = _pkg()
     with sw.Handle(0) as h:
         h.set_option("overflow_threshold", 40)
+        h.set_option("rescore_rows", rows)
         db = h.load_db(dc, do)
         out = np.zeros((2, 120), dtype=np.int32)
         h.search(qc, qo, db, sw.blosum62(), 10, 2, out=out)
